@@ -1,0 +1,329 @@
+"""Pins for liboracle's tenant definitions: closed forms, invariants, library
+routines (numpy / scipy / networkx) and brute force on tiny inputs -- never the
+oracle's own formula retyped."""
+import numpy as np
+import pytest
+
+import synth
+from synth import gen
+
+pytestmark = pytest.mark.usefixtures("oracle_lib")
+
+
+def T():
+    from oracle import tenants
+    return tenants
+
+
+# ---------------------------------------------------------------- mop
+@pytest.mark.parametrize("nconst", [0, 1, 11, 36, 37, 1000])
+def test_mop_group_dependence(nconst):
+    d = synth.preset("mop", "tiny", nconst=nconst)
+    out = T().mop(d)
+    g = np.arange(d["n"]) // d["block"]
+    ref = np.where(g < nconst, d["ina"] + d["inb"], d["ina"] - d["inb"])
+    assert np.array_equal(out, ref)
+
+
+# ---------------------------------------------------------------- stencil
+def _quad_field(nx, ny, nz):
+    z, y, x = np.meshgrid(np.arange(nz), np.arange(ny), np.arange(nx), indexing="ij")
+    return (x * x + 2 * y * y + 3 * z * z).astype(np.float32)
+
+
+def test_stencil_quadratic_closed_form():
+    """f = x^2 + 2y^2 + 3z^2: the 6-neighbour sum is 6f + 2(1+2+3), so one
+    sweep with c0 = 1/6, c1 = 1/36 gives exactly 12/36 = 1/3 inside."""
+    nx, ny, nz = 9, 7, 6
+    d = {"a0": _quad_field(nx, ny, nz), "nx": nx, "ny": ny, "nz": nz, "sweeps": 1,
+         "c0": 1.0 / 6.0, "c1": 1.0 / 36.0}
+    out = T().stencil(d)
+    assert np.allclose(out[1:-1, 1:-1, 1:-1], 1.0 / 3.0, rtol=0, atol=1e-12)
+    f = d["a0"].astype(np.float64)
+    for sl in [np.s_[0], np.s_[-1], np.s_[:, 0], np.s_[:, -1], np.s_[:, :, 0], np.s_[:, :, -1]]:
+        assert np.array_equal(out[sl], f[sl])
+
+
+def test_stencil_matches_scipy_correlate():
+    """Several sweeps vs scipy.ndimage.correlate with the 7-point kernel,
+    boundary faces held at the input values."""
+    from scipy import ndimage
+    d = synth.preset("stencil", "tiny", sweeps=4)
+    k = np.zeros((3, 3, 3))
+    k[0, 1, 1] = k[2, 1, 1] = k[1, 0, 1] = k[1, 2, 1] = k[1, 1, 0] = k[1, 1, 2] = d["c1"]
+    k[1, 1, 1] = -d["c0"]
+    a = d["a0"].astype(np.float64)
+    for _ in range(d["sweeps"]):
+        b = ndimage.correlate(a, k, mode="nearest")
+        b[0], b[-1] = a[0], a[-1]
+        b[:, 0], b[:, -1] = a[:, 0], a[:, -1]
+        b[:, :, 0], b[:, :, -1] = a[:, :, 0], a[:, :, -1]
+        a = b
+    assert np.allclose(T().stencil(d), a, rtol=1e-12, atol=1e-14)
+
+
+# ---------------------------------------------------------------- histo
+@pytest.mark.parametrize("size,over", [("tiny", {}), ("tiny", dict(bins=4096, sample_bytes=4)),
+                                       ("small", {})])
+def test_histo_bincount(size, over):
+    d = synth.preset("histo", size, **over)
+    counts, sat = T().histo(d)
+    ref = np.bincount(d["samples"].astype(np.int64), minlength=d["bins"])
+    assert np.array_equal(counts, ref)
+    assert counts.sum() == d["n"]
+    assert np.array_equal(sat, np.minimum(ref, 255))
+
+
+# ---------------------------------------------------------------- bfs
+def test_bfs_networkx():
+    import networkx as nx
+    d = synth.preset("bfs", "tiny")
+    level, depth = T().bfs(d)
+    g = nx.DiGraph()
+    g.add_nodes_from(range(d["nv"]))
+    rp, col = d["row_ptr"], d["col"]
+    for u in range(d["nv"]):
+        g.add_edges_from((u, int(w)) for w in col[rp[u]:rp[u + 1]])
+    ref = np.full(d["nv"], -1, dtype=np.int32)
+    for v, l in nx.single_source_shortest_path_length(g, d["src"]).items():
+        ref[v] = l
+    assert np.array_equal(level, ref)
+    assert depth == ref.max()
+
+
+def bfs_certificate(d, level):
+    """level[src] = 0; every edge u->v from a reached u has 0 <= level[v] <=
+    level[u] + 1; every v with level[v] > 0 has an in-edge from level[v]-1;
+    unreached vertices have no in-edge from a reached vertex."""
+    rp = d["row_ptr"].astype(np.int64)
+    col = d["col"].astype(np.int64)
+    src = np.repeat(np.arange(d["nv"]), np.diff(rp))
+    assert level[d["src"]] == 0
+    lu, lv = level[src], level[col]
+    reached = lu >= 0
+    assert np.all(lv[reached] >= 0)
+    assert np.all(lv[reached] <= lu[reached] + 1)
+    parent_ok = np.zeros(d["nv"], dtype=bool)
+    tight = reached & (lv == lu + 1)
+    parent_ok[col[tight]] = True
+    need = level > 0
+    assert np.all(parent_ok[need])
+    return True
+
+
+def test_bfs_certificate_small():
+    d = synth.preset("bfs", "small", seed=3)
+    level, _ = T().bfs(d)
+    assert bfs_certificate(d, level)
+
+
+def test_bfs_scipy():
+    from scipy.sparse import csr_matrix
+    from scipy.sparse.csgraph import shortest_path
+    d = synth.preset("bfs", "small", seed=5, src=17)
+    level, _ = T().bfs(d)
+    m = csr_matrix((np.ones(d["ne"]), d["col"], d["row_ptr"].astype(np.int64)),
+                   shape=(d["nv"], d["nv"]))
+    sp = shortest_path(m, unweighted=True, indices=d["src"])
+    ref = np.where(np.isinf(sp), -1, sp).astype(np.int32)
+    assert np.array_equal(level, ref)
+
+
+# ---------------------------------------------------------------- cutcp
+def _lattice(nx, ny, nz):
+    k, j, i = np.meshgrid(np.arange(nz), np.arange(ny), np.arange(nx), indexing="ij")
+    return np.stack([i.ravel(), j.ravel(), k.ravel()], axis=1).astype(np.int32)
+
+
+def test_cutcp_single_atom_closed_form():
+    h, c, e = 0.5, 3.0, 1.0
+    atoms = np.array([[2.25, 1.75, 2.0, 0.8]], dtype=np.float32)
+    d = {"atoms": atoms, "natoms": 1, "h": h, "cutoff": c, "excl": e}
+    pts = _lattice(11, 11, 11)
+    v = T().cutcp_points(d, pts)
+    p = pts.astype(np.float64) * h
+    r = np.linalg.norm(p - atoms[0, :3].astype(np.float64), axis=1)
+    ref = np.where(r < c, 0.8 / r * (1 - r * r / (c * c)) ** 2, 0.0)
+    ref = np.where(r < e, 0.0, ref)
+    assert np.allclose(v, ref, rtol=1e-6, atol=1e-12)  # fp32 inputs, fp64 terms
+    assert np.count_nonzero(v) > 10 and np.count_nonzero(ref == 0) > 10
+
+
+def test_cutcp_cutoff_boundary_is_zero():
+    """An atom exactly at r = c contributes nothing (membership is r^2 < c^2,
+    and the switch (1 - r^2/c^2)^2 vanishes there anyway)."""
+    d = {"atoms": np.array([[3.0, 0.0, 0.0, 1.0]], dtype=np.float32), "natoms": 1,
+         "h": 0.5, "cutoff": 3.0, "excl": 0.5}
+    assert T().cutcp_points(d, np.array([[0, 0, 0]]))[0] == 0.0
+    assert T().cutcp_points(d, np.array([[1, 0, 0]]))[0] > 0.0
+
+
+def test_cutcp_mirror_charges_cancel():
+    """+q and -q mirrored across the plane x = 8: V = 0 on that plane."""
+    atoms = np.array([[5.5, 4.0, 4.25, 0.7], [10.5, 4.0, 4.25, -0.7]], dtype=np.float32)
+    d = {"atoms": atoms, "natoms": 2, "h": 0.5, "cutoff": 6.0, "excl": 1.0}
+    pts = _lattice(33, 17, 17)
+    pts = pts[pts[:, 0] == 16]
+    v = T().cutcp_points(d, pts)
+    assert np.all(v == 0.0)
+
+
+def test_cutcp_superposition_and_scaling():
+    d = synth.preset("cutcp", "tiny", seed=2)
+    a = d["atoms"]
+    # keep only points far from every atom so no exclusion triggers
+    pts = _lattice(d["nx"], d["ny"], d["nz"])
+    p = pts.astype(np.float32) * np.float32(d["h"])
+    dist2 = ((p[:, None, :] - a[None, :, :3]) ** 2).sum(-1).min(1)
+    pts = pts[dist2 > 1.5]
+    half = len(a) // 2
+    da = dict(d, atoms=np.ascontiguousarray(a[:half]), natoms=half)
+    db = dict(d, atoms=np.ascontiguousarray(a[half:]), natoms=len(a) - half)
+    v = T().cutcp_points(d, pts)
+    va = T().cutcp_points(da, pts)
+    vb = T().cutcp_points(db, pts)
+    assert np.allclose(v, va + vb, rtol=1e-12, atol=1e-12)
+    a2 = a.copy()
+    a2[:, 3] *= 2
+    v2 = T().cutcp_points(dict(d, atoms=a2), pts)
+    assert np.allclose(v2, 2 * v, rtol=1e-12, atol=1e-12)
+
+
+def test_cutcp_full_lattice_matches_points():
+    d = synth.preset("cutcp", "tiny", seed=1)
+    full = T().cutcp(d)
+    pts = _lattice(d["nx"], d["ny"], d["nz"])
+    assert np.array_equal(full.ravel(), T().cutcp_points(d, pts))
+
+
+def test_cutcp_binning_is_consistent():
+    """The input layout (atoms sorted by cell, CSR offsets) lists every atom
+    in the cell that contains it."""
+    d = synth.preset("cutcp", "small", seed=4)
+    n1 = d["ncell_1d"]
+    cs = d["cell_start"]
+    assert cs[0] == 0 and cs[-1] == d["natoms"]
+    a = d["atoms"]
+    for c in range(n1 ** 3):
+        x, y, z = c % n1, (c // n1) % n1, c // (n1 * n1)
+        blk = a[cs[c]:cs[c + 1], :3]
+        lo = np.array([x, y, z], dtype=np.float32) * np.float32(d["cell"])
+        assert np.all(blk >= lo) and np.all(blk < lo + np.float32(d["cell"]) + 1e-6)
+    assert abs(a[:, 3].sum()) < 1e-2  # neutral molecules
+
+
+# ---------------------------------------------------------------- tpacf
+def _tpacf_numpy(d):
+    """float32 numpy: elementwise products/sums round to nearest without FMA,
+    same association as the definition; bins via np.searchsorted."""
+    binb = d["binb"]
+    asc = binb[::-1]
+    nb = len(binb) + 1
+
+    def hist(p, q, upper):
+        dot = (p[0][:, None] * q[0][None, :] + p[1][:, None] * q[1][None, :]) + \
+            p[2][:, None] * q[2][None, :]
+        assert dot.dtype == np.float32
+        if upper:
+            iu = np.triu_indices(p.shape[1], k=1)
+            dot = dot[iu]
+        b = len(binb) - np.searchsorted(asc, dot.ravel(), side="right")
+        return np.bincount(b, minlength=nb).astype(np.uint64)
+
+    dd = hist(d["data"], d["data"], True)
+    rr = sum(hist(r, r, True) for r in d["rand"])
+    dr = sum(hist(d["data"], r, False) for r in d["rand"])
+    return dd, rr, dr
+
+
+def test_tpacf_numpy_float32():
+    d = synth.preset("tpacf", "tiny")
+    dd, rr, dr = T().tpacf(d)
+    rdd, rrr, rdr = _tpacf_numpy(d)
+    assert np.array_equal(dd, rdd) and np.array_equal(rr, rrr) and np.array_equal(dr, rdr)
+
+
+def test_tpacf_pair_counts():
+    d = synth.preset("tpacf", "small", seed=9)
+    dd, rr, dr = T().tpacf(d)
+    n, s = d["npts"], d["nsets"]
+    assert dd.sum() == n * (n - 1) // 2
+    assert rr.sum() == s * n * (n - 1) // 2
+    assert dr.sum() == s * n * n
+
+
+def test_tpacf_identical_points_in_bin0():
+    """Coincident points (angle 0) land in the smallest-angle bin; antipodal
+    points in the largest."""
+    p = np.array([[1.0, 1.0, -1.0], [0.0, 0.0, 0.0], [0.0, 0.0, 0.0]], dtype=np.float32)
+    d = {"data": p, "rand": p[None].copy(), "npts": 3, "nsets": 1, "binb": gen.tpacf_bin_edges()}
+    dd, rr, dr = T().tpacf(d)
+    assert dd[0] == 1 and dd[-1] == 2
+    assert dr[0] == 5 and dr[-1] == 4
+
+
+# ---------------------------------------------------------------- spmv
+def test_spmv_scipy():
+    from scipy.sparse import csr_matrix
+    d = synth.preset("spmv", "small", seed=1)
+    y = T().spmv(d)
+    m = csr_matrix((d["val"].astype(np.float64), d["col"], d["row_ptr"]), shape=(d["n"], d["n"]))
+    assert np.allclose(y, m @ d["x"].astype(np.float64), rtol=1e-13, atol=1e-13)
+    assert d["nnz"] == (5 * 32 - 6) ** 2  # per axis sum_i #{di: 0 <= i+di < g} = 5g - 6
+
+
+def test_spmv_identity():
+    n = 50
+    d = {"row_ptr": np.arange(n + 1, dtype=np.int32), "col": np.arange(n, dtype=np.int32),
+         "val": np.ones(n, dtype=np.float32), "x": np.linspace(-3, 3, n).astype(np.float32), "n": n}
+    assert np.array_equal(T().spmv(d), d["x"].astype(np.float64))
+
+
+# ---------------------------------------------------------------- sgemm
+def test_sgemm_numpy():
+    d = synth.preset("sgemm", "tiny")
+    c = T().sgemm(d)
+    ref = d["a"].astype(np.float64) @ d["b"].astype(np.float64).T
+    assert np.allclose(c, ref, rtol=1e-12, atol=1e-12)
+    ij = np.array([[0, 0], [199, 135], [17, 3]])
+    assert np.array_equal(T().sgemm_entries(d, ij), c[ij[:, 0], ij[:, 1]])
+
+
+def test_sgemm_identity():
+    k = 64
+    a = synth.preset("sgemm", "tiny", k=k)["a"]
+    d = {"a": a, "b": np.eye(k, dtype=np.float32), "m": a.shape[0], "n": k, "k": k}
+    assert np.array_equal(T().sgemm(d), a.astype(np.float64))
+
+
+# ---------------------------------------------------------------- mri-q
+def test_mriq_phimag_float32():
+    d = synth.preset("mriq", "tiny")
+    pm = T().mriq_phimag(d)
+    assert np.array_equal(pm, d["phir"] * d["phir"] + d["phii"] * d["phii"])
+
+
+def test_mriq_complex_exponential():
+    """Qr + i Qi = sum_k phiMag_k exp(2 pi i k.x) (numpy complex128)."""
+    d = synth.preset("mriq", "tiny")
+    pm, qr, qi = T().mriq(d)
+    x = np.stack([d["x"], d["y"], d["z"]]).astype(np.float64)
+    k = np.stack([d["kx"], d["ky"], d["kz"]]).astype(np.float64)
+    q = np.exp(2j * np.pi * (k.T @ x)).T @ pm.astype(np.float64)
+    assert np.allclose(qr, q.real, rtol=1e-10, atol=1e-10)
+    assert np.allclose(qi, q.imag, rtol=1e-10, atol=1e-10)
+
+
+def test_mriq_origin_and_dc():
+    d = synth.preset("mriq", "tiny")
+    d["x"][0] = d["y"][0] = d["z"][0] = 0.0
+    d["kx"][5] = d["ky"][5] = d["kz"][5] = 0.0
+    pm = T().mriq_phimag(d)
+    qr, qi = T().mriq_points(d, np.array([0]))
+    assert qr[0] == pytest.approx(pm.astype(np.float64).sum(), rel=1e-13)
+    assert qi[0] == 0.0
+    # numK = 1, sample at k = 0: every voxel sees Qr = phiMag, Qi = 0
+    d1 = dict(d, numk=1, kx=d["kx"][5:6].copy(), ky=d["ky"][5:6].copy(), kz=d["kz"][5:6].copy(),
+              phir=d["phir"][5:6].copy(), phii=d["phii"][5:6].copy())
+    qr, qi = T().mriq_points(d1, np.arange(50))
+    assert np.all(qr == np.float64(T().mriq_phimag(d1)[0])) and np.all(qi == 0.0)
