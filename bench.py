@@ -1,0 +1,448 @@
+#!/usr/bin/env python
+"""accelOS-on-B200 bench: fair space sharing of one GPU by concurrent tenants.
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--config c2] [--impl accel|reference]
+
+One STEP = one mix of tenant kernel-execution requests (BASELINE.json config,
+default config 2 = the paper's Fig. 2 mix bfs + cutcp + stencil + tpacf,
+PAPER.md lines 289-299) submitted together through the C ABI and run to
+completion: solver quotas + persistent dispatch (SHARED mode).  The same mix
+is also run in NATIVE mode (standard concurrent streams, Fig. 1a) for the
+"vs native streams" comparison, and every tenant alone (NATIVE) for T(a).
+
+Headline metric (BASELINE.json): unfairness (max/min slowdown), STP and ANTT
+vs native streams -> reported under "sharing".  `value` is whole-job
+throughput in mixes/s (all GPUs), device-timed with CUDA events.
+
+Multi-GPU (torchrun): every rank runs its own independent mix on its own GPU
+(no collective on the data path, PAPER.md has one accelerator; BASELINE
+config 5); ranks only barrier and gather timings; value = all mixes / max
+over ranks of the device time.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import math
+import os
+import statistics
+import sys
+import threading
+import time
+
+os.environ.setdefault("CUDA_DEVICE_MAX_CONNECTIONS", "32")
+ROOT = os.path.dirname(os.path.abspath(__file__))
+if ROOT not in sys.path:
+    sys.path.insert(0, ROOT)
+
+import numpy as np  # noqa: E402
+
+import synth  # noqa: E402
+
+METRIC = "unfairness (max/min slowdown), STP and ANTT vs native streams, 1–8 B200"
+UNIT = "mixes/s"
+
+# BASELINE.json configs -> (tenants in arrival order, preset size, seeds)
+CONFIGS = {
+    "c1": dict(tenants=["stencil", "histo"], size="small", seeds=[1, 2],
+               desc="2 tenants on 1 GPU: stencil 64^3 fp32 + histo 256K uint8"),
+    "c2": dict(tenants=["bfs", "cutcp", "stencil", "tpacf"], size="default", seeds=[3, 4, 5, 6],
+               desc="Paper Fig.2 mix: bfs + cutcp + stencil + tpacf concurrently on 1xB200"),
+}
+ALL_TENANTS = ["bfs", "cutcp", "stencil", "tpacf", "histo", "spmv", "sgemm", "mriq"]
+
+
+def c5_mix(rank: int) -> list[str]:
+    """BASELINE config 5: an ordered 4-tuple of distinct tenants per GPU, seed 100+g."""
+    r = np.random.Generator(np.random.PCG64(100 + rank))
+    return [ALL_TENANTS[i] for i in r.permutation(len(ALL_TENANTS))[:4]]
+
+
+def env_rank():
+    return (int(os.environ.get("RANK", 0)), int(os.environ.get("WORLD_SIZE", 1)),
+            int(os.environ.get("LOCAL_RANK", 0)))
+
+
+# ----------------------------------------------------------------- clocks
+class ClockSampler:
+    """NVML sampling of SM clock and throttle reasons during the timed region."""
+
+    REASONS = {0x1: "gpu_idle", 0x2: "applications_clocks_setting", 0x4: "sw_power_cap",
+               0x8: "hw_slowdown", 0x10: "sync_boost", 0x20: "sw_thermal_slowdown",
+               0x40: "hw_thermal_slowdown", 0x80: "hw_power_brake_slowdown",
+               0x100: "display_clock_setting"}
+
+    def __init__(self, device: int, period: float = 0.1):
+        self.device, self.period = device, period
+        self.samples: list[int] = []
+        self.reasons: set[str] = set()
+        self.max_mhz = None
+        self._stop = threading.Event()
+        self._t = None
+        try:
+            import pynvml
+            pynvml.nvmlInit()
+            self.nv = pynvml
+            self.h = pynvml.nvmlDeviceGetHandleByIndex(device)
+            self.max_mhz = pynvml.nvmlDeviceGetMaxClockInfo(self.h, pynvml.NVML_CLOCK_SM)
+        except Exception as e:  # noqa: BLE001
+            self.nv = None
+            self.err = str(e)
+
+    def _run(self):
+        while not self._stop.is_set():
+            try:
+                self.samples.append(self.nv.nvmlDeviceGetClockInfo(self.h, self.nv.NVML_CLOCK_SM))
+                mask = self.nv.nvmlDeviceGetCurrentClocksEventReasons(self.h)
+                for bit, name in self.REASONS.items():
+                    if mask & bit and name != "gpu_idle":
+                        self.reasons.add(name)
+            except Exception:  # noqa: BLE001
+                pass
+            time.sleep(self.period)
+
+    def __enter__(self):
+        if self.nv:
+            self._t = threading.Thread(target=self._run, daemon=True)
+            self._t.start()
+        return self
+
+    def __exit__(self, *exc):
+        self._stop.set()
+        if self._t:
+            self._t.join()
+
+    def summary(self):
+        if not self.nv:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": [], "error": self.err}
+        return {"sm_mhz": statistics.median(self.samples) if self.samples else None,
+                "sm_max_mhz": self.max_mhz, "reasons": sorted(self.reasons),
+                "samples": len(self.samples)}
+
+
+# ----------------------------------------------------------------- oracle leg
+def oracle_sample(name: str, d: dict, budget: float) -> tuple[float, str]:
+    """Time the CPU oracle on a bounded sample of one tenant request and
+    extrapolate to the whole request.  Returns (seconds for the full request,
+    description of the sample)."""
+    from oracle import tenants as O
+    t0 = time.perf_counter()
+    if name == "stencil":
+        s = max(1, min(d["sweeps"], int(budget / 0.2) or 1))
+        O.stencil(dict(d, sweeps=s))
+        dt = time.perf_counter() - t0
+        return dt * d["sweeps"] / s, f"stencil {s}/{d['sweeps']} sweeps at full size"
+    if name == "histo":
+        O.histo(d)
+        dt = time.perf_counter() - t0
+        return dt * d["iters"], f"histo 1/{d['iters']} iterations"
+    if name == "bfs":
+        O.bfs(d)
+        return time.perf_counter() - t0, "bfs full"
+    if name == "cutcp":
+        npts = d["nx"] * d["ny"] * d["nz"]
+        m = int(min(npts, max(256, budget * 2e8 / max(d["natoms"], 1))))
+        r = np.random.Generator(np.random.PCG64(0))
+        flat = r.choice(npts, m, replace=False)
+        ijk = np.stack([flat % d["nx"], (flat // d["nx"]) % d["ny"], flat // (d["nx"] * d["ny"])], 1)
+        t0 = time.perf_counter()
+        O.cutcp_points(d, ijk)
+        dt = time.perf_counter() - t0
+        return dt * npts / m, f"cutcp {m}/{npts} lattice points"
+    if name == "tpacf":
+        sub = dict(d, nsets=1, rand=np.ascontiguousarray(d["rand"][:1]))
+        O.tpacf(sub)
+        dt = time.perf_counter() - t0
+        # DD once + per set (RR + DR); the sample did DD + 1 set
+        return dt * (1 + 3 * d["nsets"]) / 4, f"tpacf DD + 1/{d['nsets']} random sets"
+    if name == "spmv":
+        O.spmv(d)
+        dt = time.perf_counter() - t0
+        return dt * d["iters"], f"spmv 1/{d['iters']} iterations"
+    if name == "sgemm":
+        m = min(d["m"], 64)
+        ij = np.stack(np.meshgrid(np.arange(m), np.arange(min(d["n"], 64)), indexing="ij"), -1).reshape(-1, 2)
+        t0 = time.perf_counter()
+        O.sgemm_entries(d, ij)
+        dt = time.perf_counter() - t0
+        return dt * d["m"] * d["n"] / len(ij), f"sgemm {len(ij)}/{d['m'] * d['n']} entries"
+    if name == "mriq":
+        m = min(d["numx"], 2048)
+        idx = np.arange(m) * (d["numx"] // m)
+        t0 = time.perf_counter()
+        O.mriq_points(d, idx)
+        dt = time.perf_counter() - t0
+        return dt * d["numx"] / m, f"mri-q {m}/{d['numx']} voxels"
+    raise KeyError(name)
+
+
+def cpu_mix_seconds(tenants, inputs, budget_per_tenant):
+    tot = 0.0
+    desc = []
+    for name in tenants:
+        s, what = oracle_sample(name, inputs[name], budget_per_tenant)
+        tot += s
+        desc.append(what)
+    return tot, "; ".join(desc)
+
+
+def make_inputs(cfg_name: str, rank: int):
+    if cfg_name == "c5":
+        tenants = c5_mix(rank)
+        size = "default"
+        seeds = [100 + rank + 7 * i for i in range(4)]
+    else:
+        c = CONFIGS[cfg_name]
+        tenants, size, seeds = c["tenants"], c["size"], c["seeds"]
+    inputs = {t: synth.preset(t, size, seed=s) for t, s in zip(tenants, seeds)}
+    return tenants, size, inputs
+
+
+def run_reference(args):
+    """--impl reference: the CPU oracle as it stands (this tier's reference
+    arm), on bounded samples of the same workload, on the host cores."""
+    rank, world, _ = env_rank()
+    if rank != 0:
+        return
+    tenants, size, inputs = make_inputs(args.config, 0)
+    from oracle import tenants as O
+    O.build()
+    for _ in range(args.warmup):
+        cpu_mix_seconds(tenants, inputs, 0.3)
+    secs = []
+    desc = ""
+    for _ in range(args.steps):
+        s, desc = cpu_mix_seconds(tenants, inputs, 0.3)
+        secs.append(s)
+    ms = 1e3 * statistics.mean(secs)
+    value = 1e3 / ms
+    cores = os.cpu_count()
+    line = {"impl": "reference", "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": args.gpus,
+            "steps": args.steps, "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True,
+            "scaling": "weak", "vs_baseline": None, "dtype": "f64", "data": "synthetic",
+            "config": {"workload": CONFIGS.get(args.config, {}).get("desc", args.config),
+                       "tenants": tenants, "size": size},
+            "cpu_baseline": {"value": value, "unit": UNIT, "cores": cores, "kind": "oracle",
+                             "sample": desc + " (extrapolated to the full requests, run serially "
+                                              "with OpenMP on all host cores)"},
+            "e2e": {"value": value, "unit": UNIT, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
+    print(json.dumps(line), flush=True)
+
+
+# ----------------------------------------------------------------- GPU leg
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=10)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--config", default="c2", choices=["c1", "c2", "c5"])
+    ap.add_argument("--impl", default="accel", choices=["accel", "reference"])
+    ap.add_argument("--calib-reps", type=int, default=5)
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--out", default=None, help="also write the JSON line here")
+    args = ap.parse_args()
+    if args.impl == "reference":
+        run_reference(args)
+        return
+
+    import torch
+    import torch.distributed as dist
+
+    from paper_conf_cgo_margiolaso16_b200 import abi
+    from paper_conf_cgo_margiolaso16_b200.jobs import make_job
+    from paper_conf_cgo_margiolaso16_b200.runtime import Accel
+
+    rank, world, local = env_rank()
+    torch.cuda.set_device(local)
+    if world > 1:
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+    cfg_name = args.config if world == 1 or args.config != "c2" else "c2"
+    tenants, size, inputs = make_inputs(cfg_name, rank)
+    dev = torch.device("cuda", local)
+    jobs = [make_job(t, inputs[t], dev) for t in tenants]
+    acc = Accel(device=local, mode=abi.MODE_SHARED)
+    flush_buf = torch.empty(256 * 1024 * 1024 // 4, dtype=torch.float32, device=dev)  # > L2 (126 MB)
+
+    def flush():
+        flush_buf.fill_(1.0)
+        torch.cuda.synchronize()
+
+    def run_group(js, mode, e2e=False, launch_events=False):
+        if acc.mode != mode:
+            acc.set_mode(mode)
+        flush()
+        acc.epoch()
+        ids = acc.submit(js, e2e=e2e, launch_events=launch_events)
+        acc.sync()
+        st = [acc.stats(i) for i in ids]
+        lt = [acc.launch_times(i, j.launches()) for i, j in zip(ids, js)] if launch_events else None
+        acc.release()
+        return st, lt
+
+    # -- correctness pass (untimed): coverage of every VG, both modes
+    with Accel(device=local, mode=abi.MODE_SHARED, verify=True) as vacc:
+        for mode in (abi.MODE_NATIVE, abi.MODE_SHARED):
+            vacc.set_mode(mode)
+            st = vacc.run(jobs)
+            assert all(s.coverage_ok == 1 for s in st), "coverage check failed"
+
+    # -- calibration: T(a) = native isolated (median), persistent isolated
+    iso_native, iso_persist, iso_launch = {}, {}, {}
+    for j in jobs:
+        for mode, store in ((abi.MODE_NATIVE, iso_native), (abi.MODE_SHARED, iso_persist)):
+            ts, lts = [], []
+            for _ in range(args.calib_reps):
+                st, lt = run_group([j], mode, launch_events=True)
+                ts.append(st[0].elapsed_ms)
+                lts.append(lt[0])
+            store[j.name] = statistics.median(ts)
+            if mode == abi.MODE_SHARED:
+                iso_launch[j.name] = lts
+    ta = [iso_native[t] for t in tenants]
+
+    def steps_loop(mode, k, e2e=False):
+        out = []
+        for _ in range(k):
+            st, lt = run_group(jobs, mode, e2e=e2e, launch_events=True)
+            out.append((st, lt))
+        return out
+
+    steps_loop(abi.MODE_SHARED, args.warmup)
+    if world > 1:
+        dist.barrier()
+    torch.cuda.synchronize()
+    with ClockSampler(local) as clk:
+        shared = steps_loop(abi.MODE_SHARED, args.steps)
+    torch.cuda.synchronize()
+    if world > 1:
+        dist.barrier()
+    steps_loop(abi.MODE_NATIVE, args.warmup)
+    native = steps_loop(abi.MODE_NATIVE, args.steps)
+    steps_loop(abi.MODE_SHARED, 1, e2e=True)
+    e2e = steps_loop(abi.MODE_SHARED, args.steps, e2e=True)
+
+    def summarize(runs):
+        mk, U, STP, ANTT, OV = [], [], [], [], []
+        for st, _ in runs:
+            mk.append(max(s.done_ms for s in st) - min(s.arrival_ms for s in st))
+            ts = [s.elapsed_ms for s in st]
+            m = abi.accel_metrics(ta, ts)
+            U.append(m.unfairness)
+            STP.append(m.stp)
+            ANTT.append(m.antt)
+            OV.append(abi.accel_overlap([float(s.first_start_ns) for s in st],
+                                        [float(s.last_end_ns) for s in st]))
+        return {"makespan_ms": mk, "U": U, "STP": STP, "ANTT": ANTT, "O": OV,
+                "ts_ms": [[s.elapsed_ms for s in st] for st, _ in runs]}
+
+    sh, na, ee = summarize(shared), summarize(native), summarize(e2e)
+    dev_ms = sum(sh["makespan_ms"])
+    e2e_ms = sum(ee["makespan_ms"])
+    nat_ms = sum(na["makespan_ms"])
+
+    # roofline of the dominant kernel: the tenant with the largest device time
+    # in the shared step; per-launch CUDA-event durations on its stream
+    works = {j.name: j.work() for j in jobs}
+    tot = {t: statistics.mean(ts[i] for ts in sh["ts_ms"]) for i, t in enumerate(tenants)}
+    roof = {}
+    peaks = json.load(open(os.path.join(ROOT, "MEASURED_PEAKS.json"))) if os.path.exists(
+        os.path.join(ROOT, "MEASURED_PEAKS.json")) else {"hbm_gbs": 6650.0, "bf16_tflops": 1590.0}
+    for i, t in enumerate(tenants):
+        w = works[t]
+        if "bytes_per_launch" not in w and "bytes" not in w and "flops" not in w:
+            continue
+        per_launch = [x for _, lt in shared for x in lt[i][w.get("skip_launches", 0):]]
+        iso = [x for lt in iso_launch[t] for x in lt[w.get("skip_launches", 0):]]
+        avg = statistics.mean(per_launch)
+        avg_iso = statistics.mean(iso)
+        if w["bound"] == "hbm":
+            b = w.get("bytes_per_launch", w.get("bytes"))
+            ach, ach_iso, peak, unit = b / avg / 1e6, b / avg_iso / 1e6, peaks["hbm_gbs"], "GB/s"
+        else:
+            f = w.get("flops_per_launch", w.get("flops"))
+            ach, ach_iso, unit = f / avg / 1e9, f / avg_iso / 1e9, "TFLOP/s"
+            peak = w.get("peak_tflops", peaks.get("bf16_tflops"))
+        roof[t] = {"bound": w["bound"], "achieved": ach, "peak": peak, "unit": unit, "frac": ach / peak,
+                   "traffic": None, "avg_launch_ms": avg, "isolated": {"achieved": ach_iso,
+                                                                      "frac": ach_iso / peak,
+                                                                      "avg_launch_ms": avg_iso}}
+    dom = max(roof, key=lambda t: tot[t]) if roof else None
+
+    launches_per_step = sum(1 + j.launches() for j in jobs)  # descriptor init + kernel launches
+    h2d = sum(j.h2d_bytes() for j in jobs)
+    d2h = sum(j.d2h_bytes() for j in jobs)
+
+    local_res = {"rank": rank, "dev_ms": dev_ms, "e2e_ms": e2e_ms, "nat_ms": nat_ms,
+                 "tenants": tenants, "sh": sh, "na": na, "clk": clk.summary()}
+    if world > 1:
+        allres = [None] * world
+        dist.all_gather_object(allres, local_res)
+    else:
+        allres = [local_res]
+
+    cpu = None
+    if rank == 0 and world == 1 and not args.no_cpu_baseline:
+        from oracle import tenants as O
+        O.build()
+        s, desc = cpu_mix_seconds(tenants, inputs, 3.0)
+        cpu = {"value": 1.0 / s, "unit": UNIT, "cores": os.cpu_count(), "kind": "oracle",
+               "sample": desc + " (extrapolated to the full requests, run serially with OpenMP "
+                                "on all host cores)"}
+
+    if rank == 0:
+        tmax = max(r["dev_ms"] for r in allres)
+        emax = max(r["e2e_ms"] for r in allres)
+        nmax = max(r["nat_ms"] for r in allres)
+        value = world * args.steps / (tmax / 1e3)
+        gm = lambda xs: math.exp(statistics.mean(math.log(x) for x in xs))  # noqa: E731
+        U_sh = gm([u for r in allres for u in r["sh"]["U"]])
+        U_na = gm([u for r in allres for u in r["na"]["U"]])
+        stp_sh = statistics.mean(u for r in allres for u in r["sh"]["STP"])
+        stp_na = statistics.mean(u for r in allres for u in r["na"]["STP"])
+        antt_sh = statistics.mean(u for r in allres for u in r["sh"]["ANTT"])
+        antt_na = statistics.mean(u for r in allres for u in r["na"]["ANTT"])
+        clocks = allres[0]["clk"]
+        line = {
+            "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": args.steps,
+            "warmup": args.warmup, "ms_per_step": tmax / args.steps, "higher_is_better": True,
+            "scaling": "weak", "vs_baseline": None, "dtype": "f32+i32", "data": "synthetic",
+            "config": {"workload": CONFIGS.get(cfg_name, {}).get("desc", "config 5 mix per GPU"),
+                       "config": cfg_name, "tenants": [r["tenants"] for r in allres] if world > 1 else tenants,
+                       "size": size, "mode": "SHARED (accelOS persistent, static quotas)",
+                       "l2": "flushed before every step (256 MiB write)",
+                       "parallelism": f"independent mix per GPU x{world}"},
+            "sharing": {
+                "unfairness_shared": U_sh, "unfairness_native": U_na,
+                "fairness_improvement": U_na / U_sh,
+                "stp_shared": stp_sh, "stp_native": stp_na, "stp_ratio": stp_sh / stp_na,
+                "antt_shared": antt_sh, "antt_native": antt_na,
+                "throughput_speedup": nmax / tmax,
+                "overlap_shared": statistics.mean(o for r in allres for o in r["sh"]["O"]),
+                "overlap_native": statistics.mean(o for r in allres for o in r["na"]["O"]),
+                "T_a_ms": dict(zip(tenants, ta)),
+                "T_s_ms_shared": dict(zip(tenants, np.mean(sh["ts_ms"], 0).tolist())),
+                "T_s_ms_native": dict(zip(tenants, np.mean(na["ts_ms"], 0).tolist())),
+                "dispatch_overhead": {t: iso_persist[t] / iso_native[t] - 1 for t in tenants},
+                "native_mixes_per_s": world * args.steps / (nmax / 1e3),
+            },
+            "e2e": {"value": world * args.steps / (emax / 1e3), "unit": UNIT,
+                    "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h},
+            "gpu_launches": launches_per_step * args.steps,
+            "roofline": dict(roof[dom], kernel=dom) if dom else None,
+            "rooflines": roof,
+            "cpu_baseline": cpu,
+            "clocks": {"sm_mhz": clocks.get("sm_mhz"), "sm_max_mhz": clocks.get("sm_max_mhz"),
+                       "reasons": clocks.get("reasons")},
+        }
+        s = json.dumps(line)
+        print(s, flush=True)
+        if args.out:
+            with open(args.out, "w") as f:
+                f.write(s + "\n")
+    acc.close()
+    if world > 1:
+        dist.destroy_process_group()
+
+
+if __name__ == "__main__":
+    main()

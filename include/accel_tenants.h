@@ -1,0 +1,144 @@
+/*
+ * accel_tenants.h -- argument structs of the built-in tenant kernels of
+ * libaccel.so (see accel_builtin_kernel).  One struct per kernel, passed as
+ * accel_launch.args; all pointers are DEVICE pointers owned by the caller.
+ *
+ * PAPER.md only names the Parboil kernels it mixes (lines 289-298, 853-860,
+ * 978-989); the definitions are the Parboil-shaped readings of DESIGN.md
+ * §Tenants.  Virtual group (VG) = one original CTA; the "grid" column is the
+ * original NDRange in VGs that the caller passes in accel_launch.grid.
+ */
+#ifndef ACCEL_TENANTS_H_
+#define ACCEL_TENANTS_H_
+
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+/* mop -- PAPER.md Fig. 8a (lines 735-746).  block 256, grid ceil(n/256).
+ * out[g] = ina[g] + inb[g] if (g / 256) < nconst else ina[g] - inb[g]. */
+typedef struct {
+  const float *ina;
+  const float *inb;
+  float *out;
+  uint32_t n;
+  uint32_t nconst;
+} accel_mop_args;
+
+/* stencil -- 7-point Jacobi, fp32, A[z][y][x] (x fastest, nx % 4 == 0).
+ * block 256 (8 warps x 32 lanes x 4 x-points), VG tile 128 x 8 x 8 (x,y,z):
+ * grid (ceil(nx/128), ceil(ny/8), ceil(nz/8)).  Launch r reads
+ * (r == 0 ? a0 : buf[(r-1)&1]) and writes buf[r&1]; after T launches the
+ * result is in buf[(T-1)&1].  Interior: c1*(6-neighbour sum) - c0*a;
+ * faces copy the input. */
+typedef struct {
+  const float *a0;
+  float *buf0;
+  float *buf1;
+  uint32_t nx, ny, nz;
+  float c0, c1;
+} accel_stencil_args;
+
+/* histo -- saturating histogram (Parboil histo main + final fused).
+ * block 256, VG = `per_vg` samples (multiple of 4096), grid ceil(n/per_vg).
+ * Launch r accumulates into hist[(r&1)*bins + b]; the VG that completes the
+ * launch (done[r] reaches the VG count) writes sat[b] = min(hist, 255) and
+ * zeroes hist[((r+1)&1)*bins ...] for launch r+1.  The request must clear
+ * hist[0..bins) and done[0..launches) first.  bins <= 4096; sample_bytes 1
+ * (u8, bins == 256) or 4 (u32). */
+typedef struct {
+  const void *samples;
+  uint32_t n;
+  uint32_t bins;
+  uint32_t sample_bytes;
+  uint32_t per_vg;
+  uint32_t *hist;  /* [2][bins] */
+  uint8_t *sat;    /* [bins]    */
+  uint32_t *done;  /* [launches] */
+} accel_histo_args;
+
+/* bfs -- level-synchronous top-down BFS on a directed CSR graph.
+ * block 256, VG = 256 frontier vertices, static grid ceil(nv/256) (upper
+ * bound; persistent CTAs read the live frontier size).  Launch l expands
+ * level l.  The request must set level[] to -1 (memset 0xFF) and count[] to 0;
+ * count has (launches + 1) entries, frontier is [2][nv]. */
+typedef struct {
+  const uint32_t *row_ptr;
+  const int32_t *col;
+  uint32_t nv;
+  uint32_t src;
+  int32_t *level;
+  int32_t *frontier;
+  uint32_t *count;
+} accel_bfs_args;
+
+/* cutcp -- cutoff Coulomb potential on the lattice h*(i,j,k).  atoms float4
+ * (x,y,z,q) sorted into ncell^3 cells of edge `cell` (cell_start CSR).
+ * block 128, VG = 8x8x8 lattice points, grid ceil(n?/8).  V[k][j][i]. */
+typedef struct {
+  const float *atoms;       /* float4[natoms] */
+  const int32_t *cell_start;
+  uint32_t ncell;
+  float cell;
+  uint32_t nx, ny, nz;
+  float h, cutoff, excl;
+  float *v;
+} accel_cutcp_args;
+
+/* tpacf -- angular two-point correlation histograms, SoA unit vectors.
+ * block 256, VG = (set s in [0, 2*nsets], 256-point block i): s == 0 -> DD,
+ * s = 1..nsets -> RR of set s-1, s = nsets+1..2*nsets -> DR of set
+ * s-nsets-1; grid (ceil(npts/256), 2*nsets+1).  dd/rr/dr u64[nedges+1],
+ * cleared by the request. */
+typedef struct {
+  const float *data;   /* [3][npts]          */
+  const float *rand;   /* [nsets][3][npts]   */
+  const float *binb;   /* [nedges] descending */
+  uint32_t npts, nsets, nedges;
+  unsigned long long *dd, *rr, *dr;
+} accel_tpacf_args;
+
+/* spmv -- y = A x, CSR fp32.  block 256, VG = 64 rows, grid ceil(n/64). */
+typedef struct {
+  const int32_t *row_ptr;
+  const int32_t *col;
+  const float *val;
+  const float *x;
+  float *y;
+  uint32_t n;
+} accel_spmv_args;
+
+/* sgemm -- C[m][n] = A[m][k] . B[n][k]^T, fp32 in/out.
+ * VG = one 128 x 128 tile of C, grid (ceil(n/128), ceil(m/128)). */
+typedef struct {
+  const float *a;
+  const float *b;
+  float *c;
+  uint32_t m, n, k;
+} accel_sgemm_args;
+
+/* mri-q ComputePhiMag: phimag = phir^2 + phii^2.  block 256, grid ceil(numk/256). */
+typedef struct {
+  const float *phir;
+  const float *phii;
+  float *phimag;
+  uint32_t numk;
+} accel_mriq_phimag_args;
+
+/* mri-q ComputeQ: Qr + iQi = sum_k phimag_k exp(2 pi i k.x).
+ * block 256, VG = 256 voxels, grid ceil(numx/256). */
+typedef struct {
+  const float *kx, *ky, *kz;
+  const float *phimag;
+  uint32_t numk;
+  uint32_t numx;
+  const float *x, *y, *z;
+  float *qr, *qi;
+} accel_mriq_q_args;
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* ACCEL_TENANTS_H_ */

@@ -1,0 +1,213 @@
+// dispatch.cuh -- device side of accelOS software work-group scheduling on sm_100a.
+//
+// PAPER.md §2.4 (lines 439-459) and Fig. 8b (lines 748-781): the original
+// work-groups of a kernel execution become virtual groups (VGs) in a Virtual
+// NDRange in device memory; a reduced set of physical work-groups runs a loop
+// in which a master work-item dequeues VG(s) atomically, the group
+// synchronises, leaves on RUN_TERMINATE, else runs the kernel body for every
+// VG in [wg_base, wg_end).  §6.2 steps 1-3 (lines 719-724): the kernel becomes
+// a plain function whose work-item built-ins (get_group_id ...) read the
+// virtual id.  §6.4 (lines 824-834): one dequeue may take several VGs.
+//
+// B200 design: the JIT transformation of §6 is replaced
+// by a compile-time C++ template.  A tenant is a struct T with
+//     using Args = <plain C struct>;  static constexpr int kThreads, kChunk;
+//     static constexpr uint32_t kDynSmem;
+//     static __device__ void body(const Args&, const VirtualBlock&, char* smem);
+// optionally  static constexpr bool kDynamicTotal = true;
+//             static __device__ uint32_t dynamic_total(const Args&, uint32_t launch_idx);
+// The body never reads blockIdx/gridDim (the `mop` test catches that), keeps
+// no state across VGs and never waits on another CTA, so the wrapper is
+// deadlock-free whatever the co-residency.
+//   accel_persistent<T>: the reduced-grid scheduling kernel (Fig. 8b dyn_sched).
+//   accel_native<T>:     the same body on the original grid (Fig. 1a baseline).
+#pragma once
+
+#include <cstdint>
+#include <type_traits>
+
+namespace accel {
+
+// Virtual NDRange of ONE launch ("Virtual Kernel Execution
+// Range which is copied to the accelerator memory").  128 B, two lines: the
+// read-mostly fields and stamps, then the hot dequeue counter on its own line.
+struct alignas(128) Desc {
+  uint32_t total;        // VGs in the original grid (static upper bound)
+  uint32_t gx, gy, gz;   // original grid shape (decode, R-disp-2)
+  uint32_t chunk;        // VGs per dequeue (§6.4)
+  uint32_t launch_idx;   // index of this launch inside its step
+  uint32_t flags;        // kFlag*
+  uint32_t total_seen;   // dynamic total as read by the CTAs (bfs)
+  uint32_t* live_quota;  // RESOLVE: CTAs with index >= *live_quota leave
+  uint32_t* coverage;    // verify: coverage[vg] += 1
+  unsigned long long t_first;  // min %globaltimer over CTA starts
+  unsigned long long t_last;   // max %globaltimer over CTA ends
+  uint32_t ctas_started; // CTAs that entered the scheduling loop
+  uint32_t alive;        // CTAs currently in the loop
+  uint32_t max_alive;    // high-water mark of `alive`
+  uint32_t pad0[3];
+  // ---- line 1: the software queue head (RUN_TERMINATE when >= total)
+  uint32_t next;
+  uint32_t pad1[31];
+};
+static_assert(sizeof(Desc) == 256, "Desc layout");
+
+enum : uint32_t { kFlagStamps = 1u, kFlagAlive = 2u };
+
+// Replacement of the OpenCL work-item built-ins (get_group_id / get_num_groups,
+// PAPER.md §6.3): what a body sees instead of blockIdx/gridDim.
+struct VirtualBlock {
+  uint32_t x, y, z;        // get_group_id(0..2)
+  uint32_t gx, gy, gz;     // get_num_groups(0..2)
+  uint32_t linear;         // x + gx*(y + gy*z)
+  uint32_t launch_idx;     // launch index inside the request step
+};
+
+__device__ __forceinline__ unsigned long long globaltimer() {
+  unsigned long long t;
+  asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
+  return t;
+}
+
+__device__ __forceinline__ uint32_t ld_volatile(const uint32_t* p) {
+  uint32_t v;
+  asm volatile("ld.volatile.global.u32 %0, [%1];" : "=r"(v) : "l"(p));
+  return v;
+}
+
+// Optional T::kMinBlocks: minimum resident CTAs per SM for __launch_bounds__,
+// applied to BOTH instantiations so native and persistent get the same
+// register budget (§6.5: the transformation must not
+// add register pressure).
+template <class T, class = void>
+struct min_blocks : std::integral_constant<int, 1> {};
+template <class T>
+struct min_blocks<T, std::void_t<decltype(T::kMinBlocks)>> : std::integral_constant<int, T::kMinBlocks> {};
+
+template <class T, class = void>
+struct has_dynamic_total : std::false_type {};
+template <class T>
+struct has_dynamic_total<T, std::void_t<decltype(T::kDynamicTotal)>>
+    : std::integral_constant<bool, T::kDynamicTotal> {};
+
+template <class T>
+__device__ __forceinline__ uint32_t vg_total(const typename T::Args& a, const Desc* d,
+                                             uint32_t launch_idx) {
+  if constexpr (has_dynamic_total<T>::value) {
+    uint32_t t = T::dynamic_total(a, launch_idx);
+    return t < d->total ? t : d->total;
+  } else {
+    return d->total;
+  }
+}
+
+__device__ __forceinline__ VirtualBlock decode(uint32_t vg, uint32_t gx, uint32_t gy,
+                                               uint32_t gz, uint32_t launch_idx) {
+  VirtualBlock b;
+  b.gx = gx; b.gy = gy; b.gz = gz;
+  b.linear = vg;
+  b.launch_idx = launch_idx;
+  if (gy == 1 && gz == 1) {   // 1-D grids: no division
+    b.x = vg; b.y = 0; b.z = 0;
+  } else {
+    const uint32_t q = vg / gx;
+    b.x = vg - q * gx;
+    b.y = q % gy;
+    b.z = q / gy;
+  }
+  return b;
+}
+
+constexpr uint32_t kTerminate = 0xffffffffu;
+
+// One dequeue by the master thread (Fig. 8b line 26 rt_sched_wgroup):
+// RESOLVE shrink first (a CTA beyond the live quota leaves without consuming),
+// then one atomicAdd of `chunk` on the queue head.
+__device__ __forceinline__ uint32_t dequeue(Desc* d, uint32_t cta, uint32_t chunk) {
+  const uint32_t* lq = d->live_quota;
+  if (lq != nullptr && cta >= ld_volatile(lq)) return kTerminate;
+  return atomicAdd(&d->next, chunk);
+}
+
+// -------------------------------------------------------------------------
+// The scheduling kernel: grid = quota n_i (1-D), block = the original block.
+// cta_base > 0 for top-up launches that join a running Virtual NDRange.
+template <class T>
+__global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
+    accel_persistent(const typename T::Args args, Desc* __restrict__ d, uint32_t cta_base) {
+  extern __shared__ __align__(128) char smem[];
+  __shared__ uint32_t s_base[2];   // double-buffered dequeue result (sd.wg_base)
+  __shared__ uint32_t s_total;
+  const uint32_t cta = cta_base + blockIdx.x;
+  const uint32_t flags = d->flags;
+  const uint32_t chunk = d->chunk;
+  const uint32_t launch_idx = d->launch_idx;
+  const uint32_t gx = d->gx, gy = d->gy, gz = d->gz;
+  uint32_t* const coverage = d->coverage;
+
+  if (threadIdx.x == 0) {  // master work-item: environment init (rt_env_init)
+    if (flags & kFlagStamps) atomicMin(&d->t_first, globaltimer());
+    const uint32_t total = vg_total<T>(args, d, launch_idx);
+    s_total = total;
+    const uint32_t b = dequeue(d, cta, chunk);
+    s_base[0] = b;
+    if (b < total && (flags & kFlagAlive)) {
+      atomicAdd(&d->ctas_started, 1u);
+      const uint32_t a = atomicAdd(&d->alive, 1u) + 1u;
+      atomicMax(&d->max_alive, a);
+    }
+  }
+  __syncthreads();
+  const uint32_t total = s_total;
+  const bool started = s_base[0] < total;
+  uint32_t buf = 0;
+  for (;;) {
+    const uint32_t base = s_base[buf];
+    if (base >= total) break;                  // RUN_TERMINATE
+    uint32_t nxt = 0;
+    if (threadIdx.x == 0) nxt = dequeue(d, cta, chunk);  // prefetch next chunk
+    const uint32_t end = min(base + chunk, total);
+    for (uint32_t vg = base; vg < end; ++vg) {
+      const VirtualBlock vb = decode(vg, gx, gy, gz, launch_idx);
+      T::body(args, vb, smem);
+      if (coverage != nullptr && threadIdx.x == 0) atomicAdd(&coverage[vg], 1u);
+      if (vg + 1 < end) __syncthreads();       // body smem reuse across VGs
+    }
+    if (threadIdx.x == 0) s_base[buf ^ 1] = nxt;
+    __syncthreads();
+    buf ^= 1;
+  }
+  if (threadIdx.x == 0) {
+    if (started && (flags & kFlagAlive)) atomicSub(&d->alive, 1u);
+    if (flags & kFlagStamps) atomicMax(&d->t_last, globaltimer());
+    if (cta == 0) d->total_seen = total;
+  }
+}
+
+// The original kernel: one CTA per VG, hardware block scheduler (Fig. 1a).
+template <class T>
+__global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
+    accel_native(const typename T::Args args, Desc* __restrict__ d, uint32_t /*unused*/) {
+  extern __shared__ __align__(128) char smem[];
+  const uint32_t flags = d->flags;
+  if (threadIdx.x == 0 && (flags & kFlagStamps)) atomicMin(&d->t_first, globaltimer());
+  VirtualBlock vb;
+  vb.x = blockIdx.x; vb.y = blockIdx.y; vb.z = blockIdx.z;
+  vb.gx = gridDim.x; vb.gy = gridDim.y; vb.gz = gridDim.z;
+  vb.linear = blockIdx.x + gridDim.x * (blockIdx.y + gridDim.y * blockIdx.z);
+  vb.launch_idx = d->launch_idx;
+  bool run = true;
+  uint32_t total = d->total;
+  if constexpr (has_dynamic_total<T>::value) {
+    total = vg_total<T>(args, d, vb.launch_idx);
+    run = vb.linear < total;
+  }
+  if (vb.linear == 0 && threadIdx.x == 0) d->total_seen = total;
+  if (run) {
+    T::body(args, vb, smem);
+    if (d->coverage != nullptr && threadIdx.x == 0) atomicAdd(&d->coverage[vb.linear], 1u);
+  }
+  if (threadIdx.x == 0 && (flags & kFlagStamps)) atomicMax(&d->t_last, globaltimer());
+}
+
+}  // namespace accel

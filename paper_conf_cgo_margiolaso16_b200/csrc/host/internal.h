@@ -1,0 +1,36 @@
+// internal.h -- interfaces between the host runtime and the device code of libaccel.
+#pragma once
+#include <cstdint>
+
+#include <cuda_runtime.h>
+
+#include "accel.h"
+
+namespace accel {
+
+struct Desc;  // csrc/device/dispatch.cuh
+
+struct InitStep {
+  uint32_t first;      // first descriptor of the step
+  uint32_t launches;   // repeat count
+  uint32_t total;      // VGs per launch (static)
+  uint32_t gx, gy, gz;
+  uint32_t chunk;
+  uint32_t cov_offset; // coverage offset of the step's first launch
+};
+
+struct InitParams {
+  Desc* d;
+  uint32_t* live_quota;   // nullptr under STATIC
+  uint32_t live_init;     // initial live quota of the main step
+  uint32_t* coverage;     // nullptr unless verify
+  uint32_t flags;
+  uint32_t n_steps;
+  InitStep steps[ACCEL_MAX_STEPS];
+};
+
+// Fill the descriptors of one request on `s` (one tiny kernel).
+cudaError_t launch_desc_init(const InitParams& p, uint32_t n_desc, cudaStream_t s);
+constexpr size_t kDescBytes = 256;
+
+}  // namespace accel

@@ -1,0 +1,674 @@
+// runtime.cpp -- host runtime of libaccel: context, kernel registry, request
+// table, the Kernel Scheduler of PAPER.md §5 (lines 647-655) and stats.
+//
+// Kernel Scheduler, restated: for every kernel execution request select the
+// number of work-groups with the resource-sharing algorithm (§3), construct the
+// Virtual NDRange in accelerator memory, change the global size to the new
+// number of work-groups keeping the work-group size and dimensions, launch.
+// Here: accel_solve() over the active requests, one descriptor per launch
+// written by a tiny kernel on the tenant's stream, then cudaLaunchKernel of
+// accel_persistent<T> with grid = quota.  NATIVE mode launches accel_native<T>
+// on the original grid instead (the standard-sharing baseline, Fig. 1a).
+#include <cuda_runtime.h>
+
+#include <algorithm>
+#include <cstdio>
+#include <cstring>
+#include <map>
+#include <memory>
+#include <mutex>
+#include <string>
+#include <vector>
+
+#include "accel.h"
+#include "internal.h"
+
+namespace {
+
+using accel::InitParams;
+using accel::kDescBytes;
+
+constexpr uint32_t kPoolSlots = 16384;      // 4 MiB of descriptors
+constexpr uint32_t kFlagStamps = 1u, kFlagAlive = 2u;  // dispatch.cuh
+
+struct Kernel {
+  std::string name;
+  const void* pfn;
+  const void* nfn;
+  dim3 block;
+  uint32_t dyn_smem;
+  uint32_t chunk;
+  uint32_t args_size;
+  int num_regs;
+  int static_smem;
+  int occ_p, occ_n;
+  uint32_t threads() const { return block.x * block.y * block.z; }
+};
+
+struct Step {
+  int kid;
+  accel_dim3 grid;
+  uint32_t total;
+  std::vector<unsigned char> args;
+  uint32_t repeat;
+  uint32_t quota;
+  uint32_t first;       // first descriptor (relative to the request's slot)
+  uint64_t cov_offset;  // coverage offset of the first launch
+};
+
+struct Request {
+  uint64_t id;
+  int tenant;
+  uint32_t flags;
+  uint32_t weight;
+  int mode;
+  std::vector<Step> steps;
+  int main_step;
+  std::vector<accel_clear> clears;
+  std::vector<accel_copy> h2d, d2h;
+  cudaEvent_t ev_arrival = nullptr, ev_done = nullptr;
+  std::vector<cudaEvent_t> ev_launch;  // ACCEL_REQ_LAUNCH_EVENTS: n_desc + 1
+  uint32_t slot = 0, n_desc = 0;
+  uint32_t* cov = nullptr;
+  uint64_t cov_elems = 0;
+  uint32_t quota_initial = 0, quota_min = 0, quota_max = 0, resolves = 0;
+  bool done = false;
+  bool fetched = false;
+  int cov_ok = -1;
+  std::vector<unsigned char> desc_host;
+};
+
+bool is_sticky(cudaError_t e) {
+  switch (e) {
+    case cudaErrorIllegalAddress:
+    case cudaErrorLaunchFailure:
+    case cudaErrorIllegalInstruction:
+    case cudaErrorMisalignedAddress:
+    case cudaErrorInvalidAddressSpace:
+    case cudaErrorInvalidPc:
+    case cudaErrorHardwareStackError:
+    case cudaErrorAssert:
+    case cudaErrorLaunchTimeout:
+    case cudaErrorECCUncorrectable:
+      return true;
+    default:
+      return false;
+  }
+}
+
+std::string g_init_error;
+
+// Host view of the device descriptor (csrc/device/dispatch.cuh accel::Desc).
+struct DescHost {
+  uint32_t total, gx, gy, gz, chunk, launch_idx, flags, total_seen;
+  uint64_t live_quota, coverage;
+  unsigned long long t_first, t_last;
+  uint32_t ctas_started, alive, max_alive;
+};
+
+}  // namespace
+
+struct accel_ctx {
+  accel_config cfg{};
+  accel_caps caps{};
+  std::mutex mu;
+  std::string err;
+  bool poisoned = false;
+  std::vector<Kernel> kernels;
+  cudaStream_t main[ACCEL_MAX_TENANTS] = {};
+  cudaStream_t topup[ACCEL_MAX_TENANTS] = {};
+  cudaStream_t ctl = nullptr;
+  cudaEvent_t epoch = nullptr;
+  bool epoch_set = false;
+  unsigned char* pool = nullptr;
+  uint32_t* quota_words = nullptr;
+  std::vector<uint8_t> slot_used;
+  std::map<uint64_t, std::unique_ptr<Request>> reqs;
+  uint64_t next_id = 1;
+  std::vector<cudaEvent_t> free_events;
+
+  int fail(int code, const std::string& msg) {
+    err = msg;
+    return code;
+  }
+  int cuda(cudaError_t e, const char* what) {
+    if (e == cudaSuccess) return ACCEL_OK;
+    err = std::string(what) + ": " + cudaGetErrorString(e);
+    if (is_sticky(e)) poisoned = true;
+    cudaGetLastError();
+    return ACCEL_ECUDA;
+  }
+  cudaError_t get_event(cudaEvent_t* ev) {
+    if (!free_events.empty()) {
+      *ev = free_events.back();
+      free_events.pop_back();
+      return cudaSuccess;
+    }
+    return cudaEventCreate(ev);
+  }
+  int64_t alloc_slots(uint32_t n) {
+    uint32_t run = 0;
+    for (uint32_t i = 0; i < kPoolSlots; ++i) {
+      run = slot_used[i] ? 0 : run + 1;
+      if (run == n) {
+        const uint32_t s = i + 1 - n;
+        std::fill(slot_used.begin() + s, slot_used.begin() + s + n, 1);
+        return s;
+      }
+    }
+    return -1;
+  }
+  void free_slots(uint32_t s, uint32_t n) { std::fill(slot_used.begin() + s, slot_used.begin() + s + n, 0); }
+  accel::Desc* desc_ptr(uint32_t slot) { return reinterpret_cast<accel::Desc*>(pool + (size_t)slot * kDescBytes); }
+};
+
+#define CK(ctx, call)                                  \
+  do {                                                 \
+    int _rc = (ctx)->cuda((call), #call);              \
+    if (_rc != ACCEL_OK) return _rc;                   \
+  } while (0)
+
+namespace {
+
+int refresh_done(accel_ctx* ctx, Request* r) {
+  if (r->done) return ACCEL_OK;
+  cudaError_t e = cudaEventQuery(r->ev_done);
+  if (e == cudaSuccess) {
+    r->done = true;
+  } else if (e != cudaErrorNotReady) {
+    return ctx->cuda(e, "cudaEventQuery");
+  }
+  return ACCEL_OK;
+}
+
+uint32_t step_quota(const accel_demand& main, uint32_t n_main, const accel_demand& st) {
+  if (st.grid_vgs == 0) return 0;
+  uint64_t m = (uint64_t)n_main * main.thr / st.thr;
+  m = std::min<uint64_t>(m, (uint64_t)n_main * main.regs / st.regs);
+  m = std::min<uint64_t>(m, (uint64_t)n_main * main.smem / st.smem);
+  m = std::min<uint64_t>(m, (uint64_t)n_main * main.cta / st.cta);
+  m = std::min<uint64_t>(m, st.grid_vgs);
+  return (uint32_t)std::max<uint64_t>(m, 1);
+}
+
+int demand_for(accel_ctx* ctx, const Step& s, uint32_t weight, accel_demand* d) {
+  const Kernel& k = ctx->kernels[s.kid];
+  return accel_demand_of(&ctx->caps, k.threads(), (uint32_t)k.num_regs,
+                         (uint32_t)(k.static_smem + k.dyn_smem), s.total, weight, d);
+}
+
+int fetch_result(accel_ctx* ctx, Request* r) {
+  if (r->fetched) return ACCEL_OK;
+  r->desc_host.resize((size_t)r->n_desc * kDescBytes);
+  CK(ctx, cudaMemcpy(r->desc_host.data(), ctx->desc_ptr(r->slot), r->desc_host.size(),
+                     cudaMemcpyDeviceToHost));
+  if (r->cov) {
+    std::vector<uint32_t> cov(r->cov_elems);
+    CK(ctx, cudaMemcpy(cov.data(), r->cov, cov.size() * sizeof(uint32_t), cudaMemcpyDeviceToHost));
+    bool ok = true;
+    for (const Step& s : r->steps)
+      for (uint32_t l = 0; l < s.repeat; ++l) {
+        const DescHost* d = reinterpret_cast<const DescHost*>(r->desc_host.data() + (size_t)(s.first + l) * kDescBytes);
+        // dynamic-total kernels (bfs) cover only the live part of the static grid
+        const uint32_t live = d->total_seen <= s.total ? d->total_seen : s.total;
+        const uint32_t* c = cov.data() + s.cov_offset + (uint64_t)l * s.total;
+        for (uint32_t v = 0; v < s.total; ++v) {
+          const uint32_t want = v < live ? 1u : 0u;
+          if (c[v] != want) ok = false;
+        }
+      }
+    r->cov_ok = ok ? 1 : 0;
+  }
+  r->fetched = true;
+  return ACCEL_OK;
+}
+
+int enqueue(accel_ctx* ctx, Request* r) {
+  const bool shared = r->mode == ACCEL_MODE_SHARED;
+  cudaStream_t s = ctx->main[r->tenant];
+  CK(ctx, ctx->get_event(&r->ev_arrival));
+  CK(ctx, ctx->get_event(&r->ev_done));
+  CK(ctx, cudaEventRecord(r->ev_arrival, s));
+  for (const accel_clear& c : r->clears) CK(ctx, cudaMemsetAsync(c.dst_device, c.value, c.bytes, s));
+  for (const accel_copy& c : r->h2d) CK(ctx, cudaMemcpyAsync(c.dst, c.src, c.bytes, cudaMemcpyHostToDevice, s));
+  if (r->cov) CK(ctx, cudaMemsetAsync(r->cov, 0, r->cov_elems * sizeof(uint32_t), s));
+  InitParams p{};
+  p.d = ctx->desc_ptr(r->slot);
+  const bool resolve = shared && ctx->cfg.policy == ACCEL_POLICY_RESOLVE;
+  p.live_quota = resolve ? ctx->quota_words + r->slot : nullptr;
+  p.live_init = r->steps[r->main_step].quota;
+  p.coverage = r->cov;
+  p.flags = kFlagStamps | (shared ? kFlagAlive : 0u);
+  p.n_steps = (uint32_t)r->steps.size();
+  for (size_t j = 0; j < r->steps.size(); ++j) {
+    const Step& st = r->steps[j];
+    const Kernel& k = ctx->kernels[st.kid];
+    p.steps[j] = accel::InitStep{st.first, st.repeat, st.total, st.grid.x, st.grid.y, st.grid.z,
+                                 k.chunk, (uint32_t)st.cov_offset};
+  }
+  CK(ctx, accel::launch_desc_init(p, r->n_desc, s));
+  const bool lev = (r->flags & ACCEL_REQ_LAUNCH_EVENTS) != 0;
+  if (lev) {
+    r->ev_launch.resize(r->n_desc + 1);
+    for (auto& ev : r->ev_launch) CK(ctx, ctx->get_event(&ev));
+  }
+  uint32_t li = 0;
+  for (const Step& st : r->steps) {
+    const Kernel& k = ctx->kernels[st.kid];
+    for (uint32_t l = 0; l < st.repeat; ++l, ++li) {
+      if (lev) CK(ctx, cudaEventRecord(r->ev_launch[li], s));
+      accel::Desc* d = ctx->desc_ptr(r->slot + st.first + l);
+      uint32_t cta_base = 0;
+      void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &cta_base};
+      const dim3 grid = shared ? dim3(st.quota, 1, 1) : dim3(st.grid.x, st.grid.y, st.grid.z);
+      CK(ctx, cudaLaunchKernel(shared ? k.pfn : k.nfn, grid, k.block, params, k.dyn_smem, s));
+    }
+  }
+  if (lev) CK(ctx, cudaEventRecord(r->ev_launch[li], s));
+  for (const accel_copy& c : r->d2h) CK(ctx, cudaMemcpyAsync(c.dst, c.src, c.bytes, cudaMemcpyDeviceToHost, s));
+  CK(ctx, cudaEventRecord(r->ev_done, s));
+  return ACCEL_OK;
+}
+
+int build_request(accel_ctx* ctx, const accel_request& in, std::unique_ptr<Request>* out) {
+  if (in.tenant < 0 || in.tenant >= ACCEL_MAX_TENANTS) return ctx->fail(ACCEL_EINVAL, "tenant out of range");
+  if (in.n_steps < 1 || in.n_steps > ACCEL_MAX_STEPS || !in.steps) return ctx->fail(ACCEL_EINVAL, "bad n_steps");
+  if ((in.n_clear && !in.clear) || (in.n_h2d && !in.h2d) || (in.n_d2h && !in.d2h))
+    return ctx->fail(ACCEL_EINVAL, "null clear/copy array");
+  auto r = std::make_unique<Request>();
+  r->tenant = in.tenant;
+  r->flags = in.flags;
+  r->weight = in.weight ? in.weight : 1;
+  r->mode = ctx->cfg.mode;
+  uint32_t n_desc = 0;
+  uint64_t cov = 0;
+  r->main_step = 0;
+  for (uint32_t j = 0; j < in.n_steps; ++j) {
+    const accel_launch& L = in.steps[j];
+    if (L.kernel_id < 0 || L.kernel_id >= (int)ctx->kernels.size()) return ctx->fail(ACCEL_EINVAL, "bad kernel_id");
+    const Kernel& k = ctx->kernels[L.kernel_id];
+    if (L.args_size != k.args_size || !L.args) return ctx->fail(ACCEL_EINVAL, "args_size mismatch for " + k.name);
+    if (L.repeat < 1) return ctx->fail(ACCEL_EINVAL, "repeat < 1");
+    const uint64_t total = (uint64_t)L.grid.x * L.grid.y * L.grid.z;
+    if (total == 0 || total >= 0x7fffffffull || L.grid.y > 65535 || L.grid.z > 65535)
+      return ctx->fail(ACCEL_EINVAL, "bad grid");
+    Step s;
+    s.kid = L.kernel_id;
+    s.grid = L.grid;
+    s.total = (uint32_t)total;
+    s.args.assign((const unsigned char*)L.args, (const unsigned char*)L.args + L.args_size);
+    s.repeat = L.repeat;
+    s.quota = s.total;
+    s.first = n_desc;
+    s.cov_offset = cov;
+    n_desc += L.repeat;
+    cov += (uint64_t)L.repeat * s.total;
+    r->steps.push_back(std::move(s));
+    if (r->steps.back().total > r->steps[r->main_step].total) r->main_step = (int)j;
+  }
+  r->n_desc = n_desc;
+  r->cov_elems = ctx->cfg.verify ? cov : 0;
+  r->clears.assign(in.clear, in.clear + in.n_clear);
+  r->h2d.assign(in.h2d, in.h2d + in.n_h2d);
+  r->d2h.assign(in.d2h, in.d2h + in.n_d2h);
+  *out = std::move(r);
+  return ACCEL_OK;
+}
+
+// Solve over active requests (arrival order) + the new ones; assign the new
+// ones' quotas (STATIC: running requests keep theirs).
+int assign_quotas(accel_ctx* ctx, std::vector<std::unique_ptr<Request>>& fresh) {
+  std::vector<Request*> order;
+  for (auto& kv : ctx->reqs) {
+    Request* r = kv.second.get();
+    int rc = refresh_done(ctx, r);
+    if (rc) return rc;
+    if (!r->done && r->mode == ACCEL_MODE_SHARED) order.push_back(r);
+  }
+  for (auto& r : fresh) order.push_back(r.get());
+  std::vector<accel_demand> ds(order.size());
+  for (size_t i = 0; i < order.size(); ++i) {
+    Request* r = order[i];
+    int rc = demand_for(ctx, r->steps[r->main_step], r->weight, &ds[i]);
+    if (rc) return ctx->fail(rc, "kernel does not fit on an SM");
+  }
+  std::vector<uint32_t> q(order.size());
+  int rc = accel_solve(&ctx->caps, ds.data(), (int32_t)ds.size(), q.data());
+  if (rc) return ctx->fail(rc, "accel_solve failed");
+  const size_t first_new = order.size() - fresh.size();
+  for (size_t i = first_new; i < order.size(); ++i) {
+    Request* r = order[i];
+    for (size_t j = 0; j < r->steps.size(); ++j) {
+      Step& s = r->steps[j];
+      if ((int)j == r->main_step) {
+        s.quota = q[i];
+      } else {
+        accel_demand dj;
+        rc = demand_for(ctx, s, r->weight, &dj);
+        if (rc) return ctx->fail(rc, "kernel does not fit on an SM");
+        s.quota = step_quota(ds[i], q[i], dj);
+      }
+    }
+    r->quota_initial = r->quota_min = r->quota_max = q[i];
+  }
+  return ACCEL_OK;
+}
+
+int submit_locked(accel_ctx* ctx, uint32_t n, const accel_request* rs, uint64_t* ids) {
+  if (ctx->poisoned) return ACCEL_ESTATE;
+  CK(ctx, cudaSetDevice(ctx->cfg.device));
+  std::vector<std::unique_ptr<Request>> fresh(n);
+  for (uint32_t i = 0; i < n; ++i) {
+    int rc = build_request(ctx, rs[i], &fresh[i]);
+    if (rc) return rc;
+  }
+  if (ctx->cfg.mode == ACCEL_MODE_SHARED) {
+    int rc = assign_quotas(ctx, fresh);
+    if (rc) return rc;
+  } else {
+    for (auto& r : fresh) r->quota_initial = r->quota_min = r->quota_max = r->steps[r->main_step].total;
+  }
+  // resources
+  for (uint32_t i = 0; i < n; ++i) {
+    Request* r = fresh[i].get();
+    const int64_t s = ctx->alloc_slots(r->n_desc);
+    if (s < 0) {
+      for (uint32_t j = 0; j < i; ++j) ctx->free_slots(fresh[j]->slot, fresh[j]->n_desc);
+      return ctx->fail(ACCEL_ENOMEM, "descriptor pool exhausted (release finished requests)");
+    }
+    r->slot = (uint32_t)s;
+    if (r->cov_elems) CK(ctx, cudaMalloc(&r->cov, r->cov_elems * sizeof(uint32_t)));
+  }
+  for (uint32_t i = 0; i < n; ++i) {
+    Request* r = fresh[i].get();
+    int rc = enqueue(ctx, r);
+    if (rc) return rc;
+    r->id = ctx->next_id++;
+    ids[i] = r->id;
+    ctx->reqs[r->id] = std::move(fresh[i]);
+  }
+  return ACCEL_OK;
+}
+
+void release_request(accel_ctx* ctx, Request* r) {
+  ctx->free_slots(r->slot, r->n_desc);
+  if (r->cov) cudaFree(r->cov);
+  if (r->ev_arrival) ctx->free_events.push_back(r->ev_arrival);
+  if (r->ev_done) ctx->free_events.push_back(r->ev_done);
+  for (cudaEvent_t ev : r->ev_launch) ctx->free_events.push_back(ev);
+}
+
+}  // namespace
+
+extern "C" {
+
+const char* accel_last_error(const accel_ctx* ctx) {
+  return ctx ? ctx->err.c_str() : g_init_error.c_str();
+}
+
+int accel_init(const accel_config* cfg, accel_ctx** out) {
+  if (!cfg || !out) return ACCEL_EINVAL;
+  if (cfg->mode != ACCEL_MODE_NATIVE && cfg->mode != ACCEL_MODE_SHARED) return ACCEL_EINVAL;
+  if (cfg->policy != ACCEL_POLICY_STATIC && cfg->policy != ACCEL_POLICY_RESOLVE) return ACCEL_EINVAL;
+  auto ctx = std::make_unique<accel_ctx>();
+  ctx->cfg = *cfg;
+  auto init_fail = [&](cudaError_t e, const char* what) {
+    g_init_error = std::string(what) + ": " + cudaGetErrorString(e);
+    return ACCEL_ECUDA;
+  };
+  cudaError_t e = cudaSetDevice(cfg->device);
+  if (e != cudaSuccess) return init_fail(e, "cudaSetDevice");
+  int sms = 0;
+  e = cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, cfg->device);
+  if (e != cudaSuccess) return init_fail(e, "cudaDeviceGetAttribute");
+  ctx->caps = cfg->caps;
+  if (ctx->caps.sms <= 0) ctx->caps.sms = sms;
+  for (int t = 0; t < ACCEL_MAX_TENANTS; ++t) {
+    if ((e = cudaStreamCreateWithFlags(&ctx->main[t], cudaStreamNonBlocking)) != cudaSuccess)
+      return init_fail(e, "cudaStreamCreate");
+    if ((e = cudaStreamCreateWithFlags(&ctx->topup[t], cudaStreamNonBlocking)) != cudaSuccess)
+      return init_fail(e, "cudaStreamCreate");
+  }
+  if ((e = cudaStreamCreateWithFlags(&ctx->ctl, cudaStreamNonBlocking)) != cudaSuccess)
+    return init_fail(e, "cudaStreamCreate");
+  if ((e = cudaEventCreate(&ctx->epoch)) != cudaSuccess) return init_fail(e, "cudaEventCreate");
+  if ((e = cudaMalloc(&ctx->pool, (size_t)kPoolSlots * kDescBytes)) != cudaSuccess)
+    return init_fail(e, "cudaMalloc(pool)");
+  if ((e = cudaMalloc(&ctx->quota_words, (size_t)kPoolSlots * sizeof(uint32_t))) != cudaSuccess)
+    return init_fail(e, "cudaMalloc(quota)");
+  ctx->slot_used.assign(kPoolSlots, 0);
+  *out = ctx.release();
+  return ACCEL_OK;
+}
+
+int accel_finalize(accel_ctx* ctx) {
+  if (!ctx) return ACCEL_OK;
+  cudaSetDevice(ctx->cfg.device);
+  for (auto& kv : ctx->reqs) {
+    if (kv.second->ev_done) cudaEventSynchronize(kv.second->ev_done);
+    release_request(ctx, kv.second.get());
+  }
+  ctx->reqs.clear();
+  for (cudaEvent_t ev : ctx->free_events) cudaEventDestroy(ev);
+  for (int t = 0; t < ACCEL_MAX_TENANTS; ++t) {
+    if (ctx->main[t]) cudaStreamDestroy(ctx->main[t]);
+    if (ctx->topup[t]) cudaStreamDestroy(ctx->topup[t]);
+  }
+  if (ctx->ctl) cudaStreamDestroy(ctx->ctl);
+  if (ctx->epoch) cudaEventDestroy(ctx->epoch);
+  if (ctx->pool) cudaFree(ctx->pool);
+  if (ctx->quota_words) cudaFree(ctx->quota_words);
+  delete ctx;
+  return ACCEL_OK;
+}
+
+int accel_set_mode(accel_ctx* ctx, int32_t mode, int32_t policy) {
+  if (!ctx) return ACCEL_EINVAL;
+  std::lock_guard<std::mutex> g(ctx->mu);
+  if (ctx->poisoned) return ACCEL_ESTATE;
+  if (mode != ACCEL_MODE_NATIVE && mode != ACCEL_MODE_SHARED) return ctx->fail(ACCEL_EINVAL, "bad mode");
+  if (policy != ACCEL_POLICY_STATIC && policy != ACCEL_POLICY_RESOLVE) return ctx->fail(ACCEL_EINVAL, "bad policy");
+  for (auto& kv : ctx->reqs) {
+    int rc = refresh_done(ctx, kv.second.get());
+    if (rc) return rc;
+    if (!kv.second->done) return ctx->fail(ACCEL_EINVAL, "requests still running");
+  }
+  ctx->cfg.mode = mode;
+  ctx->cfg.policy = policy;
+  return ACCEL_OK;
+}
+
+int accel_kernel_register(accel_ctx* ctx, const accel_kernel_desc* d, int32_t* kernel_id) {
+  if (!ctx || !d || !kernel_id || !d->persistent_fn || !d->native_fn) return ACCEL_EINVAL;
+  std::lock_guard<std::mutex> g(ctx->mu);
+  if (ctx->poisoned) return ACCEL_ESTATE;
+  CK(ctx, cudaSetDevice(ctx->cfg.device));
+  Kernel k;
+  k.name = d->name ? d->name : "?";
+  k.pfn = d->persistent_fn;
+  k.nfn = d->native_fn;
+  k.block = dim3(d->block.x, d->block.y ? d->block.y : 1, d->block.z ? d->block.z : 1);
+  k.dyn_smem = d->dyn_smem;
+  k.chunk = d->chunk ? d->chunk : 1;
+  k.args_size = d->args_size;
+  cudaFuncAttributes a;
+  CK(ctx, cudaFuncGetAttributes(&a, k.pfn));
+  if ((int)k.threads() > a.maxThreadsPerBlock) return ctx->fail(ACCEL_ENOFIT, "block larger than the kernel allows");
+  k.num_regs = d->regs > 0 ? d->regs : a.numRegs;
+  k.static_smem = (int)a.sharedSizeBytes;
+  for (const void* fn : {k.pfn, k.nfn}) {
+    if (k.dyn_smem > 48 * 1024)
+      CK(ctx, cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)k.dyn_smem));
+    // one carveout for every tenant so CTAs of different kernels can share an SM
+    CK(ctx, cudaFuncSetAttribute(fn, cudaFuncAttributePreferredSharedMemoryCarveout, 100));
+  }
+  CK(ctx, cudaOccupancyMaxActiveBlocksPerMultiprocessor(&k.occ_p, k.pfn, (int)k.threads(), k.dyn_smem));
+  CK(ctx, cudaOccupancyMaxActiveBlocksPerMultiprocessor(&k.occ_n, k.nfn, (int)k.threads(), k.dyn_smem));
+  accel_demand dem;
+  int rc = accel_demand_of(&ctx->caps, k.threads(), (uint32_t)k.num_regs,
+                           (uint32_t)(k.static_smem + k.dyn_smem), 1, 1, &dem);
+  if (rc) return ctx->fail(rc, "one CTA of " + k.name + " fits on no SM");
+  ctx->kernels.push_back(k);
+  *kernel_id = (int32_t)ctx->kernels.size() - 1;
+  return ACCEL_OK;
+}
+
+int accel_kernel_info_get(accel_ctx* ctx, int32_t kernel_id, accel_kernel_info* out) {
+  if (!ctx || !out) return ACCEL_EINVAL;
+  std::lock_guard<std::mutex> g(ctx->mu);
+  if (kernel_id < 0 || kernel_id >= (int)ctx->kernels.size()) return ctx->fail(ACCEL_EINVAL, "bad kernel_id");
+  const Kernel& k = ctx->kernels[kernel_id];
+  accel_demand dem;
+  int rc = accel_demand_of(&ctx->caps, k.threads(), (uint32_t)k.num_regs,
+                           (uint32_t)(k.static_smem + k.dyn_smem), 1, 1, &dem);
+  if (rc) return rc;
+  out->thr = dem.thr;
+  out->regs = dem.regs;
+  out->smem = dem.smem;
+  out->cta = dem.cta;
+  out->num_regs = k.num_regs;
+  out->static_smem = k.static_smem;
+  out->occ_persistent = k.occ_p;
+  out->occ_native = k.occ_n;
+  return ACCEL_OK;
+}
+
+int accel_submit_group(accel_ctx* ctx, uint32_t n, const accel_request* rs, uint64_t* ids) {
+  if (!ctx || (n && (!rs || !ids))) return ACCEL_EINVAL;
+  std::lock_guard<std::mutex> g(ctx->mu);
+  return submit_locked(ctx, n, rs, ids);
+}
+
+int accel_submit(accel_ctx* ctx, const accel_request* r, uint64_t* id) {
+  return accel_submit_group(ctx, 1, r, id);
+}
+
+int accel_sync(accel_ctx* ctx, uint64_t request_id) {
+  if (!ctx) return ACCEL_EINVAL;
+  std::lock_guard<std::mutex> g(ctx->mu);
+  if (ctx->poisoned) return ACCEL_ESTATE;
+  CK(ctx, cudaSetDevice(ctx->cfg.device));
+  std::vector<Request*> todo;
+  if (request_id == ACCEL_ALL) {
+    for (auto& kv : ctx->reqs) todo.push_back(kv.second.get());
+  } else {
+    auto it = ctx->reqs.find(request_id);
+    if (it == ctx->reqs.end()) return ctx->fail(ACCEL_EINVAL, "unknown request");
+    todo.push_back(it->second.get());
+  }
+  for (Request* r : todo) {
+    if (!r->done) {
+      CK(ctx, cudaEventSynchronize(r->ev_done));
+      r->done = true;
+    }
+  }
+  bool cov_bad = false;
+  for (Request* r : todo) {
+    int rc = fetch_result(ctx, r);
+    if (rc) return rc;
+    if (r->cov_ok == 0) cov_bad = true;
+  }
+  if (cov_bad) return ctx->fail(ACCEL_ECOVERAGE, "a virtual group did not run exactly once");
+  return ACCEL_OK;
+}
+
+int accel_epoch(accel_ctx* ctx) {
+  if (!ctx) return ACCEL_EINVAL;
+  std::lock_guard<std::mutex> g(ctx->mu);
+  if (ctx->poisoned) return ACCEL_ESTATE;
+  CK(ctx, cudaSetDevice(ctx->cfg.device));
+  CK(ctx, cudaEventRecord(ctx->epoch, ctx->ctl));
+  ctx->epoch_set = true;
+  return ACCEL_OK;
+}
+
+int accel_stats(accel_ctx* ctx, uint64_t request_id, accel_req_stats* out) {
+  if (!ctx || !out) return ACCEL_EINVAL;
+  std::lock_guard<std::mutex> g(ctx->mu);
+  if (ctx->poisoned) return ACCEL_ESTATE;
+  auto it = ctx->reqs.find(request_id);
+  if (it == ctx->reqs.end()) return ctx->fail(ACCEL_EINVAL, "unknown request");
+  Request* r = it->second.get();
+  int rc = refresh_done(ctx, r);
+  if (rc) return rc;
+  if (!r->done) return ACCEL_ENOTREADY;
+  rc = fetch_result(ctx, r);
+  if (rc) return rc;
+  std::memset(out, 0, sizeof(*out));
+  CK(ctx, cudaEventElapsedTime(&out->elapsed_ms, r->ev_arrival, r->ev_done));
+  if (ctx->epoch_set) {
+    CK(ctx, cudaEventElapsedTime(&out->arrival_ms, ctx->epoch, r->ev_arrival));
+    CK(ctx, cudaEventElapsedTime(&out->done_ms, ctx->epoch, r->ev_done));
+  }
+  unsigned long long first = ~0ull, last = 0;
+  uint32_t max_ctas = 0, launches = 0, vgs = 0;
+  for (uint32_t i = 0; i < r->n_desc; ++i) {
+    const DescHost* d = reinterpret_cast<const DescHost*>(r->desc_host.data() + (size_t)i * kDescBytes);
+    first = std::min(first, d->t_first);
+    last = std::max(last, d->t_last);
+    max_ctas = std::max(max_ctas, d->max_alive);
+    vgs += d->total;
+    ++launches;
+  }
+  out->first_start_ns = first;
+  out->last_end_ns = last;
+  out->vgs_total = vgs;
+  out->launches = launches;
+  out->quota_initial = r->quota_initial;
+  out->quota_min = r->quota_min;
+  out->quota_max = r->quota_max;
+  out->resolves = r->resolves;
+  out->max_ctas = max_ctas;
+  out->coverage_ok = r->cov_ok;
+  out->mode = r->mode;
+  return ACCEL_OK;
+}
+
+int accel_launch_times(accel_ctx* ctx, uint64_t request_id, float* ms_out, uint32_t n, uint32_t* n_out) {
+  if (!ctx || (n && !ms_out) || !n_out) return ACCEL_EINVAL;
+  std::lock_guard<std::mutex> g(ctx->mu);
+  if (ctx->poisoned) return ACCEL_ESTATE;
+  auto it = ctx->reqs.find(request_id);
+  if (it == ctx->reqs.end()) return ctx->fail(ACCEL_EINVAL, "unknown request");
+  Request* r = it->second.get();
+  int rc = refresh_done(ctx, r);
+  if (rc) return rc;
+  if (!r->done) return ACCEL_ENOTREADY;
+  if (r->ev_launch.empty()) return ctx->fail(ACCEL_EINVAL, "request had no ACCEL_REQ_LAUNCH_EVENTS");
+  const uint32_t m = std::min<uint32_t>(n, r->n_desc);
+  for (uint32_t i = 0; i < m; ++i)
+    CK(ctx, cudaEventElapsedTime(&ms_out[i], r->ev_launch[i], r->ev_launch[i + 1]));
+  *n_out = m;
+  return ACCEL_OK;
+}
+
+int accel_release(accel_ctx* ctx, uint64_t request_id) {
+  if (!ctx) return ACCEL_EINVAL;
+  std::lock_guard<std::mutex> g(ctx->mu);
+  for (auto it = ctx->reqs.begin(); it != ctx->reqs.end();) {
+    Request* r = it->second.get();
+    if (request_id != ACCEL_ALL && it->first != request_id) {
+      ++it;
+      continue;
+    }
+    int rc = refresh_done(ctx, r);
+    if (rc) return rc;
+    if (!r->done) {
+      if (request_id != ACCEL_ALL) return ctx->fail(ACCEL_EINVAL, "request still running");
+      ++it;
+      continue;
+    }
+    release_request(ctx, r);
+    it = ctx->reqs.erase(it);
+  }
+  return ACCEL_OK;
+}
+
+int accel_tenant_stream(accel_ctx* ctx, int32_t tenant, void** main_stream, void** topup_stream) {
+  if (!ctx || tenant < 0 || tenant >= ACCEL_MAX_TENANTS) return ACCEL_EINVAL;
+  if (main_stream) *main_stream = ctx->main[tenant];
+  if (topup_stream) *topup_stream = ctx->topup[tenant];
+  return ACCEL_OK;
+}
+
+}  // extern "C"

@@ -1,0 +1,218 @@
+// solver.cpp -- host share solver (accel_solve / accel_demand_of).
+//
+// PAPER.md §3 (lines 483-542): per kernel i the work-groups allowed by threads,
+// local memory and registers are x_i = T/(K w_i), y_i = L/(K m_i),
+// z_i = R/(K r_i); the quota is their minimum; being Diophantine the result
+// may be conservative, and a greedy heuristic adds work-groups across the
+// kernels until the resources saturate.  B200 readings (DESIGN.md
+// R-solver-1..9): floors; CTA slots as a fourth resource; warp/SMSP register
+// allocation and reserved/rounded shared memory in the demand vector; a
+// per-SM packing check F after the closed form; class-symmetric decrement and
+// greedy so identical kernels get identical quotas.  Must agree exactly with
+// the oracle (tests/test_solver_parity.py).
+#include <algorithm>
+#include <cstdint>
+#include <vector>
+
+#include "accel.h"
+
+namespace {
+
+struct Caps {
+  int64_t sms, thr, regs, smem, ctas;
+  static constexpr int64_t kSmsp = 4;
+  static constexpr int64_t kRegGran = 256;
+  static constexpr int64_t kSmemGran = 128;
+  static constexpr int64_t kSmemReserved = 1024;
+  static constexpr int64_t kMaxSmemPerCta = 232448;
+  static constexpr int64_t kMaxRegsPerThread = 255;
+  int64_t regs_per_smsp() const { return regs / kSmsp; }
+};
+
+Caps caps_of(const accel_caps* c) {
+  Caps k{148, 2048, 65536, 233472, 32};
+  if (c) {
+    if (c->sms > 0) k.sms = c->sms;
+    if (c->thr_per_sm > 0) k.thr = c->thr_per_sm;
+    if (c->regs_per_sm > 0) k.regs = c->regs_per_sm;
+    if (c->smem_per_sm > 0) k.smem = c->smem_per_sm;
+    if (c->ctas_per_sm > 0) k.ctas = c->ctas_per_sm;
+  }
+  return k;
+}
+
+int64_t cdiv(int64_t a, int64_t b) { return (a + b - 1) / b; }
+
+struct Req {
+  int64_t thr, regs, smem, cta, g, w;
+  int64_t warps() const { return thr / 32; }
+  int64_t rpw() const { return regs / warps(); }
+  bool same(const Req& o) const {
+    return thr == o.thr && regs == o.regs && smem == o.smem && cta == o.cta && g == o.g && w == o.w;
+  }
+};
+
+bool valid(const Req& r, const Caps& c) {
+  if (r.thr <= 0 || r.thr % 32 || r.thr > c.thr || r.cta != 1 || r.w <= 0) return false;
+  if (r.regs <= 0 || r.regs % r.warps() || r.rpw() % Caps::kRegGran) return false;
+  if (cdiv(r.warps(), Caps::kSmsp) * r.rpw() > c.regs_per_smsp()) return false;
+  if (r.smem <= 0 || r.smem > c.smem) return false;
+  return true;
+}
+
+// F(n): breadth-first placement with rotating remainders, per-SM sums and the
+// sub-partition register packing (least-loaded start, round-robin warps).
+bool feasible(const std::vector<Req>& rs, const std::vector<int64_t>& n, const Caps& c) {
+  const size_t k = rs.size();
+  std::vector<int64_t> q(k), rem(k), off(k);
+  int64_t o = 0;
+  for (size_t i = 0; i < k; ++i) {
+    q[i] = n[i] / c.sms;
+    rem[i] = n[i] % c.sms;
+    off[i] = o;
+    o = (o + rem[i]) % c.sms;
+  }
+  std::vector<int64_t> cnt(k), last(k, -1);
+  bool have_last = false;
+  for (int64_t sm = 0; sm < c.sms; ++sm) {
+    for (size_t i = 0; i < k; ++i) {
+      // SM `sm` gets an extra CTA of kernel i iff (sm - off_i) mod S < rem_i
+      const int64_t rel = ((sm - off[i]) % c.sms + c.sms) % c.sms;
+      cnt[i] = q[i] + (rel < rem[i] ? 1 : 0);
+    }
+    if (have_last && cnt == last) continue;  // identical SM load: same verdict
+    last = cnt;
+    have_last = true;
+    int64_t thr = 0, ctas = 0, smem = 0;
+    int64_t sp[Caps::kSmsp] = {0, 0, 0, 0};
+    for (size_t i = 0; i < k; ++i) {
+      thr += cnt[i] * rs[i].thr;
+      ctas += cnt[i] * rs[i].cta;
+      smem += cnt[i] * rs[i].smem;
+      const int64_t w = rs[i].warps(), rpw = rs[i].rpw();
+      for (int64_t t = 0; t < cnt[i]; ++t) {
+        int start = 0;
+        for (int s = 1; s < Caps::kSmsp; ++s)
+          if (sp[s] < sp[start]) start = s;
+        for (int64_t x = 0; x < w; ++x) sp[(start + x) % Caps::kSmsp] += rpw;
+      }
+    }
+    if (thr > c.thr || ctas > c.ctas || smem > c.smem) return false;
+    for (int s = 0; s < Caps::kSmsp; ++s)
+      if (sp[s] > c.regs_per_smsp()) return false;
+  }
+  return true;
+}
+
+// a/b < c/d for positive denominators, exact
+bool frac_less(__int128 a, __int128 b, __int128 c, __int128 d) { return a * d < c * b; }
+
+// dominant share of a request holding n CTAs: max_r n*d_r/(S*cap_r) as (num, den)
+void dominant(const Req& r, int64_t n, const Caps& c, __int128* num, __int128* den) {
+  const __int128 cand[4][2] = {{(__int128)n * r.thr, (__int128)c.sms * c.thr},
+                               {(__int128)n * r.regs, (__int128)c.sms * c.regs},
+                               {(__int128)n * r.smem, (__int128)c.sms * c.smem},
+                               {(__int128)n * r.cta, (__int128)c.sms * c.ctas}};
+  *num = cand[0][0];
+  *den = cand[0][1];
+  for (int i = 1; i < 4; ++i)
+    if (frac_less(*num, *den, cand[i][0], cand[i][1])) {
+      *num = cand[i][0];
+      *den = cand[i][1];
+    }
+}
+
+}  // namespace
+
+extern "C" int accel_demand_of(const accel_caps* caps, uint32_t block_threads, uint32_t regs_per_thread,
+                               uint32_t smem_bytes, uint32_t grid_vgs, uint32_t weight,
+                               accel_demand* out) {
+  if (!out || block_threads == 0) return ACCEL_EINVAL;
+  const Caps c = caps_of(caps);
+  const int64_t warps = cdiv(block_threads, 32);
+  const int64_t rpw = cdiv(32 * (int64_t)regs_per_thread, Caps::kRegGran) * Caps::kRegGran;
+  const int64_t smem = cdiv((int64_t)smem_bytes + Caps::kSmemReserved, Caps::kSmemGran) * Caps::kSmemGran;
+  if (32 * warps > c.thr || (int64_t)smem_bytes > Caps::kMaxSmemPerCta ||
+      (int64_t)regs_per_thread > Caps::kMaxRegsPerThread ||
+      cdiv(warps, Caps::kSmsp) * rpw > c.regs_per_smsp() || smem > c.smem)
+    return ACCEL_ENOFIT;
+  out->thr = (uint32_t)(32 * warps);
+  out->regs = (uint32_t)(rpw * warps);
+  out->smem = (uint32_t)smem;
+  out->cta = 1;
+  out->grid_vgs = grid_vgs;
+  out->weight = weight ? weight : 1;
+  return ACCEL_OK;
+}
+
+extern "C" int accel_solve(const accel_caps* caps, const accel_demand* d, int32_t k, uint32_t* quota_out) {
+  if (k < 0 || (k > 0 && (!d || !quota_out))) return ACCEL_EINVAL;
+  const Caps c = caps_of(caps);
+  std::vector<Req> rs(k);
+  for (int i = 0; i < k; ++i) {
+    rs[i] = Req{d[i].thr, d[i].regs, d[i].smem, d[i].cta, d[i].grid_vgs, d[i].weight ? d[i].weight : 1};
+    if (!valid(rs[i], c)) return ACCEL_ENOFIT;
+  }
+  // classes of identical requests, in order of first arrival
+  std::vector<std::vector<int>> cls;
+  for (int i = 0; i < k; ++i) {
+    bool placed = false;
+    for (auto& m : cls)
+      if (rs[m[0]].same(rs[i])) {
+        m.push_back(i);
+        placed = true;
+        break;
+      }
+    if (!placed) cls.push_back({i});
+  }
+  // closed form on device totals (weights scale the share)
+  int64_t W = 0;
+  for (auto& r : rs)
+    if (r.g > 0) W += r.w;
+  std::vector<int64_t> n(k, 0);
+  for (int i = 0; i < k; ++i) {
+    const Req& r = rs[i];
+    if (r.g == 0) continue;
+    const int64_t x = (c.sms * c.thr * r.w) / (W * r.thr);
+    const int64_t z = (c.sms * c.regs * r.w) / (W * r.regs);
+    const int64_t y = (c.sms * c.smem * r.w) / (W * r.smem);
+    const int64_t s = (c.sms * c.ctas * r.w) / (W * r.cta);
+    n[i] = std::max<int64_t>(1, std::min({x, y, z, s, r.g}));
+  }
+  // decrement whole classes with the largest dominant share until F holds
+  while (!feasible(rs, n, c)) {
+    int best = -1;
+    __int128 bn = 0, bd = 1;
+    for (size_t ci = 0; ci < cls.size(); ++ci) {
+      const int i = cls[ci][0];
+      if (n[i] <= 1) continue;
+      __int128 num, den;
+      dominant(rs[i], n[i], c, &num, &den);
+      if (best < 0 || !frac_less(num, den, bn, bd)) {  // >= : later class wins ties
+        best = (int)ci;
+        bn = num;
+        bd = den;
+      }
+    }
+    if (best < 0) break;  // 1 CTA each does not pack (tiny devices only)
+    for (int i : cls[best]) n[i] -= 1;
+  }
+  // class-symmetric greedy fill
+  for (;;) {
+    bool accepted = false;
+    for (auto& m : cls) {
+      bool room = true;
+      for (int i : m)
+        if (n[i] + 1 > rs[i].g) room = false;
+      if (!room) continue;
+      for (int i : m) n[i] += 1;
+      if (feasible(rs, n, c))
+        accepted = true;
+      else
+        for (int i : m) n[i] -= 1;
+    }
+    if (!accepted) break;
+  }
+  for (int i = 0; i < k; ++i) quota_out[i] = (uint32_t)n[i];
+  return ACCEL_OK;
+}

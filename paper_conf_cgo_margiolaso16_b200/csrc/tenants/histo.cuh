@@ -1,0 +1,88 @@
+// histo -- saturating histogram (Parboil "histo" main + final fused; PAPER.md
+// names "histo final" / "hist inter" at line 979).
+//
+// One VG = `per_vg` samples read with 16-B vector loads (coalesced, HBM-bound),
+// counted into a shared-memory private histogram with shared atomics, then
+// flushed (non-zero bins only) with global atomics into hist[r&1].  The VG that
+// completes launch r (done[r] counter, threadfence reduction) runs the "final"
+// step: sat[b] = min(hist, 255), and zeroes the other half of hist for the
+// next launch.  No cross-CTA waiting: the last finisher does the tail work.
+#pragma once
+#include "../device/dispatch.cuh"
+#include "accel_tenants.h"
+
+namespace accel {
+
+struct Histo {
+  using Args = accel_histo_args;
+  static constexpr int kThreads = 256;
+  static constexpr uint32_t kChunk = 1;
+  static constexpr int kMinBlocks = 6;    // <= 40 regs in both modes
+  static constexpr uint32_t kMaxBins = 4096;
+  static constexpr uint32_t kDynSmem = kMaxBins * sizeof(uint32_t);  // 16 KB
+
+  static __device__ __forceinline__ void count4(uint32_t* h, uint32_t w, uint32_t sb) {
+    if (sb == 1) {
+#pragma unroll
+      for (int k = 0; k < 4; ++k) atomicAdd(&h[(w >> (8 * k)) & 0xffu], 1u);
+    } else {
+      atomicAdd(&h[w], 1u);
+    }
+  }
+
+  static __device__ __forceinline__ void body(const Args& a, const VirtualBlock& vb, char* smem) {
+    uint32_t* h = reinterpret_cast<uint32_t*>(smem);
+    __shared__ bool s_last;
+    const uint32_t bins = a.bins;
+    const uint32_t r = vb.launch_idx;
+    for (uint32_t b = threadIdx.x; b < bins; b += kThreads) h[b] = 0u;
+    __syncthreads();
+
+    const uint32_t sb = a.sample_bytes;
+    const uint64_t lo = (uint64_t)vb.linear * a.per_vg;
+    const uint64_t hi = (lo + a.per_vg < (uint64_t)a.n) ? lo + a.per_vg : (uint64_t)a.n;
+    const char* base = reinterpret_cast<const char*>(a.samples);
+    // 16-B vectors fully inside [lo, hi): per_vg is a multiple of 4096 so lo
+    // is 16-B aligned for both sample sizes.
+    const uint64_t per_vec = 16 / sb;
+    const uint64_t nvec = (hi - lo) / per_vec;
+    const uint4* v = reinterpret_cast<const uint4*>(base + lo * sb);
+    for (uint64_t i = threadIdx.x; i < nvec; i += kThreads) {
+      const uint4 w = __ldcs(v + i);   // streamed once: evict-first
+      count4(h, w.x, sb);
+      count4(h, w.y, sb);
+      count4(h, w.z, sb);
+      count4(h, w.w, sb);
+    }
+    for (uint64_t i = lo + nvec * per_vec + threadIdx.x; i < hi; i += kThreads) {
+      const uint32_t s = sb == 1 ? (uint32_t)reinterpret_cast<const uint8_t*>(base)[i]
+                                 : reinterpret_cast<const uint32_t*>(base)[i];
+      atomicAdd(&h[s], 1u);
+    }
+    __syncthreads();
+    uint32_t* gh = a.hist + (r & 1u) * bins;
+    for (uint32_t b = threadIdx.x; b < bins; b += kThreads) {
+      const uint32_t c = h[b];
+      if (c) atomicAdd(&gh[b], c);
+    }
+    // final step by the VG that completes launch r
+    __threadfence();
+    __syncthreads();
+    if (threadIdx.x == 0) {
+      const uint32_t nvg = vb.gx * vb.gy * vb.gz;
+      s_last = atomicAdd(&a.done[r], 1u) == nvg - 1;
+    }
+    __syncthreads();
+    if (s_last) {
+      __threadfence();
+      uint32_t* other = a.hist + ((r + 1u) & 1u) * bins;
+      for (uint32_t b = threadIdx.x; b < bins; b += kThreads) {
+        const uint32_t c = __ldcg(gh + b);
+        a.sat[b] = (uint8_t)(c > 255u ? 255u : c);
+        other[b] = 0u;
+      }
+    }
+  }
+};
+
+}  // namespace accel

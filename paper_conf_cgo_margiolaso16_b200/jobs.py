@@ -1,0 +1,207 @@
+"""Tenant jobs: device buffers + the accel_request a tenant submits.
+
+Argument marshalling only.  Each Job uploads its seeded inputs (from `synth`)
+into device memory owned by PyTorch, allocates outputs / scratch, and
+describes its kernel execution request as steps of built-in kernels (names of
+include/accel_tenants.h) -- the computation itself runs in libaccel.so.
+
+A Job is one *request* in the sense of PAPER.md §7.2 (lines 853-860: "kernel
+execution requests"); iterative Parboil codes submit their whole launch
+sequence as one request (DESIGN.md R-job-1).
+"""
+from __future__ import annotations
+
+import ctypes as C
+from dataclasses import dataclass, field
+
+import numpy as np
+import torch
+
+from . import abi
+
+
+def _dev(a: np.ndarray, device) -> torch.Tensor:
+    a = np.ascontiguousarray(a)
+    if a.dtype == np.uint32:
+        a = a.view(np.int32)
+    elif a.dtype == np.uint64:
+        a = a.view(np.int64)
+    return torch.from_numpy(a).to(device)
+
+
+def _np(t: torch.Tensor, dtype) -> np.ndarray:
+    return t.detach().cpu().numpy().view(dtype)
+
+
+def _cdiv(a: int, b: int) -> int:
+    return -(-a // b)
+
+
+@dataclass
+class Step:
+    kernel: str
+    grid: tuple[int, int, int]
+    args: C.Structure
+    repeat: int = 1
+
+
+@dataclass
+class Job:
+    """Base class.  Subclasses fill `inputs` (device tensors the e2e path
+    copies from host), `steps`, `clears` and `outputs`."""
+    name: str = "job"
+    device: torch.device = field(default_factory=lambda: torch.device("cuda"))
+
+    def __post_init__(self):
+        self.inputs: dict[str, torch.Tensor] = {}
+        self.out: dict[str, torch.Tensor] = {}
+        self.steps: list[Step] = []
+        self.clears: list[tuple[torch.Tensor, int]] = []
+        self._pinned_in: dict[str, torch.Tensor] = {}
+        self._pinned_out: dict[str, torch.Tensor] = {}
+
+    # ---- e2e: host buffers ----------------------------------------------
+    def pin_host(self) -> None:
+        """Pinned host copies of the inputs (sources of the per-step H2D) and
+        pinned output buffers (destinations of the D2H)."""
+        for k, t in self.inputs.items():
+            h = torch.empty(t.shape, dtype=t.dtype, pin_memory=True)
+            h.copy_(t.cpu())
+            self._pinned_in[k] = h
+        for k, t in self.output_tensors().items():
+            self._pinned_out[k] = torch.empty(t.shape, dtype=t.dtype, pin_memory=True)
+
+    def h2d_bytes(self) -> int:
+        return sum(t.numel() * t.element_size() for t in self.inputs.values())
+
+    def d2h_bytes(self) -> int:
+        return sum(t.numel() * t.element_size() for t in self.output_tensors().values())
+
+    def output_tensors(self) -> dict[str, torch.Tensor]:
+        return dict(self.out)
+
+    # ---- the request ------------------------------------------------------
+    def request(self, kernel_ids: dict[str, int], tenant: int, e2e: bool = False,
+                weight: int = 1, flags: int = 0) -> abi.accel_request:
+        steps = (abi.accel_launch * len(self.steps))()
+        keep = []
+        for i, s in enumerate(self.steps):
+            steps[i] = abi.accel_launch(kernel_ids[s.kernel], abi.accel_dim3(*s.grid),
+                                        C.cast(C.pointer(s.args), C.c_void_p), C.sizeof(s.args), s.repeat)
+            keep.append(s.args)
+        clears = (abi.accel_clear * max(1, len(self.clears)))()
+        for i, (t, v) in enumerate(self.clears):
+            clears[i] = abi.accel_clear(t.data_ptr(), v, t.numel() * t.element_size())
+        h2d = (abi.accel_copy * max(1, len(self.inputs)))()
+        d2h = (abi.accel_copy * max(1, len(self.out)))()
+        nh = nd = 0
+        if e2e:
+            if not self._pinned_in:
+                self.pin_host()
+            for k, t in self.inputs.items():
+                h = self._pinned_in[k]
+                h2d[nh] = abi.accel_copy(t.data_ptr(), h.data_ptr(), t.numel() * t.element_size())
+                nh += 1
+            for k, t in self.output_tensors().items():
+                h = self._pinned_out[k]
+                d2h[nd] = abi.accel_copy(h.data_ptr(), t.data_ptr(), t.numel() * t.element_size())
+                nd += 1
+        req = abi.accel_request(tenant, flags, weight, len(self.steps), steps, len(self.clears), clears,
+                                nh, h2d, nd, d2h)
+        req._keep = (steps, clears, h2d, d2h, keep)  # keep ctypes buffers alive until submit
+        return req
+
+    def launches(self) -> int:
+        return sum(s.repeat for s in self.steps)
+
+    def kernels(self) -> list[str]:
+        return sorted({s.kernel for s in self.steps})
+
+    def result(self) -> dict[str, np.ndarray]:
+        raise NotImplementedError
+
+    def host_result(self) -> dict[str, np.ndarray]:
+        """Outputs as read back by the e2e D2H copies."""
+        raise NotImplementedError
+
+    # algorithmic work of one request, for roofline figures
+    def work(self) -> dict:
+        return {}
+
+
+class MopJob(Job):
+    def __init__(self, d: dict, device="cuda"):
+        super().__init__(name="mop", device=torch.device(device))
+        self.n, self.block = d["n"], d["block"]
+        assert self.block == 256
+        self.inputs = {"ina": _dev(d["ina"], self.device), "inb": _dev(d["inb"], self.device)}
+        self.out = {"out": torch.empty(self.n, dtype=torch.float32, device=self.device)}
+        self.args = abi.accel_mop_args(self.inputs["ina"].data_ptr(), self.inputs["inb"].data_ptr(),
+                                       self.out["out"].data_ptr(), self.n, d["nconst"])
+        self.steps = [Step("mop", (_cdiv(self.n, 256), 1, 1), self.args, 1)]
+
+    def result(self):
+        return {"out": _np(self.out["out"], np.float32)}
+
+    def work(self):
+        return {"bytes": 12 * self.n, "bound": "hbm"}
+
+
+class StencilJob(Job):
+    TX, TY, TZ = 128, 8, 8
+
+    def __init__(self, d: dict, device="cuda"):
+        super().__init__(name="stencil", device=torch.device(device))
+        self.nx, self.ny, self.nz, self.sweeps = d["nx"], d["ny"], d["nz"], d["sweeps"]
+        if self.nx % 4:
+            raise ValueError("stencil needs nx % 4 == 0 (16-B rows)")
+        n = self.nx * self.ny * self.nz
+        self.inputs = {"a0": _dev(d["a0"].ravel(), self.device)}
+        self.buf = [torch.empty(n, dtype=torch.float32, device=self.device) for _ in range(2)]
+        self.out = {"a": self.buf[(self.sweeps - 1) & 1]}
+        self.args = abi.accel_stencil_args(self.inputs["a0"].data_ptr(), self.buf[0].data_ptr(),
+                                           self.buf[1].data_ptr(), self.nx, self.ny, self.nz,
+                                           d["c0"], d["c1"])
+        grid = (_cdiv(self.nx, self.TX), _cdiv(self.ny, self.TY), _cdiv(self.nz, self.TZ))
+        self.steps = [Step("stencil", grid, self.args, self.sweeps)]
+
+    def result(self):
+        return {"a": _np(self.out["a"], np.float32).reshape(self.nz, self.ny, self.nx)}
+
+    def work(self):
+        pts = self.nx * self.ny * self.nz
+        return {"bytes": 8 * pts * self.sweeps, "bytes_per_launch": 8 * pts, "bound": "hbm",
+                "launches": self.sweeps}
+
+
+class HistoJob(Job):
+    def __init__(self, d: dict, device="cuda"):
+        super().__init__(name="histo", device=torch.device(device))
+        self.n, self.bins, self.iters, self.sb = d["n"], d["bins"], d["iters"], d["sample_bytes"]
+        assert self.bins <= 4096 and (self.sb == 4 or self.bins == 256)
+        self.per_vg = 4096 if self.sb == 1 else 16384
+        self.inputs = {"samples": _dev(d["samples"], self.device)}
+        self.hist = torch.zeros(2 * self.bins, dtype=torch.int32, device=self.device)
+        self.sat = torch.zeros(self.bins, dtype=torch.uint8, device=self.device)
+        self.done = torch.zeros(self.iters, dtype=torch.int32, device=self.device)
+        last = (self.iters - 1) & 1
+        self.out = {"counts": self.hist[last * self.bins:(last + 1) * self.bins], "sat": self.sat}
+        self.args = abi.accel_histo_args(self.inputs["samples"].data_ptr(), self.n, self.bins, self.sb,
+                                         self.per_vg, self.hist.data_ptr(), self.sat.data_ptr(),
+                                         self.done.data_ptr())
+        self.clears = [(self.hist, 0), (self.done, 0)]
+        self.steps = [Step("histo", (_cdiv(self.n, self.per_vg), 1, 1), self.args, self.iters)]
+
+    def result(self):
+        return {"counts": _np(self.out["counts"], np.uint32), "sat": _np(self.sat, np.uint8)}
+
+    def work(self):
+        b = self.n * self.sb + 4 * self.bins
+        return {"bytes": b * self.iters, "bytes_per_launch": b, "bound": "hbm", "launches": self.iters}
+
+
+JOBS = {"mop": MopJob, "stencil": StencilJob, "histo": HistoJob}
+
+
+def make_job(name: str, d: dict, device="cuda") -> Job:
+    return JOBS[name](d, device)

@@ -1,0 +1,72 @@
+"""Per-tenant isolated timing: NATIVE vs SHARED (persistent, K=1) at a preset
+size, per-launch CUDA-event times, achieved bandwidth / throughput.
+
+    python scripts/isolated.py [--size default] [--reps 5] tenant ...
+"""
+import argparse
+import json
+import os
+import statistics
+import sys
+
+os.environ.setdefault("CUDA_DEVICE_MAX_CONNECTIONS", "32")
+sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+
+import torch  # noqa: E402
+
+import synth  # noqa: E402
+from paper_conf_cgo_margiolaso16_b200 import abi  # noqa: E402
+from paper_conf_cgo_margiolaso16_b200.jobs import make_job  # noqa: E402
+from paper_conf_cgo_margiolaso16_b200.runtime import Accel  # noqa: E402
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("tenants", nargs="+")
+    ap.add_argument("--size", default="default")
+    ap.add_argument("--reps", type=int, default=5)
+    ap.add_argument("--chunk1", action="store_true")
+    args = ap.parse_args()
+    acc = Accel(0)
+    flush = torch.empty(64 * 1024 * 1024, dtype=torch.float32, device="cuda")
+    out = {}
+    for t in args.tenants:
+        d = synth.preset(t, args.size, seed=1)
+        job = make_job(t, d)
+        res = {}
+        for mode, name in ((abi.MODE_NATIVE, "native"), (abi.MODE_SHARED, "persistent")):
+            acc.set_mode(mode)
+            el, lt, q = [], [], 0
+            for _ in range(args.reps + 1):
+                flush.fill_(1)
+                torch.cuda.synchronize()
+                ids = acc.submit([job], launch_events=True)
+                acc.sync()
+                s = acc.stats(ids[0])
+                el.append(s.elapsed_ms)
+                lt.append(acc.launch_times(ids[0], job.launches()))
+                q = s.quota_initial
+                acc.release()
+            el, lt = el[1:], lt[1:]
+            w = job.work()
+            per = [x for l in lt for x in l]
+            r = {"elapsed_ms": statistics.median(el), "launch_ms_mean": statistics.mean(per),
+                 "launch_ms_min": min(per), "quota": q}
+            if w.get("bound") == "hbm":
+                b = w.get("bytes_per_launch", w.get("bytes"))
+                r["GBps_mean"] = b / r["launch_ms_mean"] / 1e6
+            elif "flops" in w or "flops_per_launch" in w:
+                f = w.get("flops_per_launch", w.get("flops"))
+                r["TFLOPs_mean"] = f / r["launch_ms_mean"] / 1e9
+            res[name] = r
+        res["overhead"] = res["persistent"]["elapsed_ms"] / res["native"]["elapsed_ms"] - 1
+        info = acc.kernel_info(job.steps[0].kernel)
+        res["regs"] = info.num_regs
+        res["occ"] = [info.occ_native, info.occ_persistent]
+        out[t] = res
+        print(t, json.dumps(res), flush=True)
+    acc.close()
+
+
+if __name__ == "__main__":
+    main()

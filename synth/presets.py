@@ -21,7 +21,7 @@ PRESETS: dict[str, dict[str, dict]] = {
         "default": dict(n=1 << 26, block=256),
     },
     "stencil": {
-        "tiny": dict(nx=70, ny=21, nz=19, sweeps=3),
+        "tiny": dict(nx=72, ny=21, nz=19, sweeps=3),
         "small": dict(nx=64, ny=64, nz=64, sweeps=100),
         "default": dict(nx=512, ny=512, nz=64, sweeps=100),
     },

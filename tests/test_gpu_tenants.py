@@ -1,0 +1,181 @@
+"""GPU parity: every tenant through the C ABI, NATIVE and SHARED (persistent)
+modes, against the CPU oracle -- bit-exact for integer work, within the north
+star's 1e-4 (R-tol-1) for fp32 -- plus native == persistent bit-exact and the
+per-VG coverage counters (every virtual group exactly once)."""
+import numpy as np
+import pytest
+
+import synth
+from tests.gpu_util import assert_close_fp32
+
+pytestmark = pytest.mark.gpu
+
+
+@pytest.fixture(scope="module")
+def acc():
+    import torch
+    if not torch.cuda.is_available():
+        pytest.skip("no GPU")
+    from paper_conf_cgo_margiolaso16_b200 import abi
+    from paper_conf_cgo_margiolaso16_b200.runtime import Accel
+    a = Accel(device=0, mode=abi.MODE_SHARED, verify=True)
+    yield a
+    a.close()
+
+
+# small solver caps force few persistent CTAs -> many VGs per CTA
+TINY_CAPS = (2, 2048, 65536, 233472, 32)
+
+
+@pytest.fixture(scope="module")
+def acc_tiny_caps():
+    import torch
+    if not torch.cuda.is_available():
+        pytest.skip("no GPU")
+    from paper_conf_cgo_margiolaso16_b200 import abi
+    from paper_conf_cgo_margiolaso16_b200.runtime import Accel
+    a = Accel(device=0, mode=abi.MODE_SHARED, verify=True, caps=abi.accel_caps(*TINY_CAPS))
+    yield a
+    a.close()
+
+
+def run_modes(acc, job_factory):
+    """Run the same job NATIVE then SHARED; return (native_result, shared_result, stats)."""
+    from paper_conf_cgo_margiolaso16_b200 import abi
+    out = {}
+    st = {}
+    for mode in (abi.MODE_NATIVE, abi.MODE_SHARED):
+        acc.set_mode(mode)
+        job = job_factory()
+        s = acc.run([job])[0]
+        assert s.coverage_ok == 1
+        out[mode] = job.result()
+        st[mode] = s
+    acc.set_mode(abi.MODE_SHARED)
+    return out[abi.MODE_NATIVE], out[abi.MODE_SHARED], st
+
+
+def same(a: dict, b: dict):
+    for k in a:
+        assert np.array_equal(a[k], b[k]), k
+
+
+# ---------------------------------------------------------------- mop
+@pytest.mark.parametrize("nconst", [0, 1, 8, 11, 16, 36, 37])
+def test_mop(acc_tiny_caps, oracle_lib, nconst):
+    from paper_conf_cgo_margiolaso16_b200.jobs import MopJob
+    d = synth.preset("mop", "tiny", nconst=nconst)
+    nat, sh, st = run_modes(acc_tiny_caps, lambda: MopJob(d))
+    ref = oracle_lib.mop(d)
+    assert np.array_equal(nat["out"], ref)
+    assert np.array_equal(sh["out"], ref)
+    assert st[1].quota_initial < 37  # fewer persistent CTAs than VGs
+
+
+def test_mop_small_fullcaps(acc, oracle_lib):
+    from paper_conf_cgo_margiolaso16_b200.jobs import MopJob
+    d = synth.preset("mop", "small")
+    nat, sh, st = run_modes(acc, lambda: MopJob(d))
+    ref = oracle_lib.mop(d)
+    assert np.array_equal(nat["out"], ref) and np.array_equal(sh["out"], ref)
+
+
+# ---------------------------------------------------------------- stencil
+@pytest.mark.parametrize("size,over", [("tiny", {}), ("tiny", dict(nx=132, ny=9, nz=17, sweeps=2)),
+                                       ("small", dict(sweeps=10))])
+def test_stencil(acc_tiny_caps, oracle_lib, size, over):
+    from paper_conf_cgo_margiolaso16_b200.jobs import StencilJob
+    d = synth.preset("stencil", size, **over)
+    nat, sh, _ = run_modes(acc_tiny_caps, lambda: StencilJob(d))
+    same(nat, sh)
+    assert_close_fp32(sh["a"], oracle_lib.stencil(d), what="stencil")
+
+
+def test_stencil_default_sampled(acc, oracle_lib):
+    """BASELINE size (512x512x64, 100 sweeps) in the bench's launch
+    configuration; the oracle at full size is ~1.7e9 point-sweeps of plain C,
+    so compare a handful of whole planes computed by the oracle on a z-slab
+    that contains every point whose value can reach them (light cone)."""
+    from paper_conf_cgo_margiolaso16_b200.jobs import StencilJob
+    d = synth.preset("stencil", "default", sweeps=12)
+    job = StencilJob(d)
+    acc.run([job])
+    got = job.result()["a"]
+    # planes z in [20, 24): depend on z in [20-12, 24+12) only
+    zlo, zhi, T = 8, 36, d["sweeps"]
+    slab = dict(d, a0=np.ascontiguousarray(d["a0"][zlo:zhi]), nz=zhi - zlo)
+    ref = oracle_lib.stencil(slab)
+    assert_close_fp32(got[20:24], ref[20 - zlo:24 - zlo], what="stencil default")
+
+
+# ---------------------------------------------------------------- histo
+@pytest.mark.parametrize("size,over", [("tiny", {}), ("tiny", dict(bins=4096, sample_bytes=4)),
+                                       ("small", {}), ("small", dict(n=(1 << 18) + 13, iters=3))])
+def test_histo(acc_tiny_caps, oracle_lib, size, over):
+    from paper_conf_cgo_margiolaso16_b200.jobs import HistoJob
+    d = synth.preset("histo", size, **over)
+    nat, sh, _ = run_modes(acc_tiny_caps, lambda: HistoJob(d))
+    counts, sat = oracle_lib.histo(d)
+    for r in (nat, sh):
+        assert np.array_equal(r["counts"], counts)
+        assert np.array_equal(r["sat"], sat)
+
+
+def test_histo_default(acc, oracle_lib):
+    from paper_conf_cgo_margiolaso16_b200.jobs import HistoJob
+    d = synth.preset("histo", "default", iters=3)
+    nat, sh, _ = run_modes(acc, lambda: HistoJob(d))
+    counts, sat = oracle_lib.histo(d)
+    assert np.array_equal(sh["counts"], counts) and np.array_equal(nat["counts"], counts)
+    assert np.array_equal(sh["sat"], sat)
+
+
+# ---------------------------------------------------------------- mixes
+def test_config1_mix_both_orders(acc, oracle_lib):
+    """BASELINE config 1: stencil 64^3 + histo 256K u8, submitted together."""
+    from paper_conf_cgo_margiolaso16_b200 import abi
+    from paper_conf_cgo_margiolaso16_b200.jobs import HistoJob, StencilJob
+    ds = synth.preset("stencil", "small", seed=1, sweeps=20)
+    dh = synth.preset("histo", "small", seed=2)
+    ref_s = oracle_lib.stencil(ds)
+    ref_h = oracle_lib.histo(dh)
+    for mode in (abi.MODE_NATIVE, abi.MODE_SHARED):
+        acc.set_mode(mode)
+        for order in ((0, 1), (1, 0)):
+            jobs = [StencilJob(ds), HistoJob(dh)]
+            st = acc.run([jobs[i] for i in order])
+            assert all(s.coverage_ok == 1 for s in st)
+            assert_close_fp32(jobs[0].result()["a"], ref_s)
+            assert np.array_equal(jobs[1].result()["counts"], ref_h[0])
+            if mode == abi.MODE_SHARED:
+                # two concurrent requests share the device: quotas sum within it
+                assert sum(s.quota_initial for s in st) <= 148 * 8
+    acc.set_mode(abi.MODE_SHARED)
+
+
+def test_e2e_host_buffers(acc, oracle_lib):
+    """The request's own H2D/D2H copies (host pinned buffers) give the same result."""
+    import torch
+    from paper_conf_cgo_margiolaso16_b200.jobs import HistoJob
+    d = synth.preset("histo", "small", seed=7)
+    job = HistoJob(d)
+    job.pin_host()
+    job.inputs["samples"].zero_()  # the H2D copy must restore it
+    torch.cuda.synchronize()
+    acc.run([job], e2e=True)
+    counts, _ = oracle_lib.histo(d)
+    assert np.array_equal(job._pinned_out["counts"].numpy().view(np.uint32), counts)
+
+
+def test_quota_matches_occupancy_for_single_tenant(acc):
+    """K = 1: quota = min(G, SMs x cudaOccupancyMaxActiveBlocksPerMultiprocessor)."""
+    import torch
+    from paper_conf_cgo_margiolaso16_b200.jobs import StencilJob
+    d = synth.preset("stencil", "default", sweeps=1)
+    job = StencilJob(d)
+    st = acc.run([job])[0]
+    info = acc.kernel_info("stencil")
+    sms = torch.cuda.get_device_properties(0).multi_processor_count
+    g = int(np.prod(job.steps[0].grid))
+    assert st.quota_initial == min(g, sms * info.occ_persistent)
+    assert info.occ_persistent == info.occ_native
