@@ -238,6 +238,8 @@ def main():
     ap.add_argument("--config", default="c2", choices=["c1", "c2", "c5"])
     ap.add_argument("--impl", default="accel", choices=["accel", "reference"])
     ap.add_argument("--calib-reps", type=int, default=5)
+    ap.add_argument("--policy", default="resolve", choices=["resolve", "static"],
+                    help="SHARED-mode policy of the timed (headline) run; the other is reported too")
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--out", default=None, help="also write the JSON line here")
     args = ap.parse_args()
@@ -267,9 +269,14 @@ def main():
         flush_buf.fill_(1.0)
         torch.cuda.synchronize()
 
-    def run_group(js, mode, e2e=False, launch_events=False):
-        if acc.mode != mode:
-            acc.set_mode(mode)
+    POL = {"resolve": abi.POLICY_RESOLVE, "static": abi.POLICY_STATIC}
+    head_pol = POL[args.policy]
+    other_pol = POL["static" if args.policy == "resolve" else "resolve"]
+
+    def run_group(js, mode, e2e=False, launch_events=False, policy=None):
+        policy = head_pol if policy is None else policy
+        if acc.mode != mode or acc.policy != policy:
+            acc.set_mode(mode, policy)
         flush()
         acc.epoch()
         ids = acc.submit(js, e2e=e2e, launch_events=launch_events)
@@ -300,10 +307,10 @@ def main():
                 iso_launch[j.name] = lts
     ta = [iso_native[t] for t in tenants]
 
-    def steps_loop(mode, k, e2e=False):
+    def steps_loop(mode, k, e2e=False, policy=None):
         out = []
         for _ in range(k):
-            st, lt = run_group(jobs, mode, e2e=e2e, launch_events=True)
+            st, lt = run_group(jobs, mode, e2e=e2e, launch_events=True, policy=policy)
             out.append((st, lt))
         return out
 
@@ -318,6 +325,8 @@ def main():
         dist.barrier()
     steps_loop(abi.MODE_NATIVE, args.warmup)
     native = steps_loop(abi.MODE_NATIVE, args.steps)
+    steps_loop(abi.MODE_SHARED, 1, policy=other_pol)
+    other = steps_loop(abi.MODE_SHARED, args.steps, policy=other_pol)
     steps_loop(abi.MODE_SHARED, 1, e2e=True)
     e2e = steps_loop(abi.MODE_SHARED, args.steps, e2e=True)
 
@@ -335,7 +344,7 @@ def main():
         return {"makespan_ms": mk, "U": U, "STP": STP, "ANTT": ANTT, "O": OV,
                 "ts_ms": [[s.elapsed_ms for s in st] for st, _ in runs]}
 
-    sh, na, ee = summarize(shared), summarize(native), summarize(e2e)
+    sh, na, ee, ot = summarize(shared), summarize(native), summarize(e2e), summarize(other)
     dev_ms = sum(sh["makespan_ms"])
     e2e_ms = sum(ee["makespan_ms"])
     nat_ms = sum(na["makespan_ms"])
@@ -373,7 +382,9 @@ def main():
     d2h = sum(j.d2h_bytes() for j in jobs)
 
     local_res = {"rank": rank, "dev_ms": dev_ms, "e2e_ms": e2e_ms, "nat_ms": nat_ms,
-                 "tenants": tenants, "sh": sh, "na": na, "clk": clk.summary()}
+                 "oth_ms": sum(ot["makespan_ms"]), "tenants": tenants, "sh": sh, "na": na, "ot": ot,
+                 "quotas": [[s.quota_initial, s.quota_min, s.quota_max, s.resolves] for s in shared[-1][0]],
+                 "clk": clk.summary()}
     if world > 1:
         allres = [None] * world
         dist.all_gather_object(allres, local_res)
@@ -401,6 +412,17 @@ def main():
         stp_na = statistics.mean(u for r in allres for u in r["na"]["STP"])
         antt_sh = statistics.mean(u for r in allres for u in r["sh"]["ANTT"])
         antt_na = statistics.mean(u for r in allres for u in r["na"]["ANTT"])
+        omax = max(r["oth_ms"] for r in allres)
+        other_name = "static" if args.policy == "resolve" else "resolve"
+        other_sum = {
+            "policy": other_name,
+            "unfairness": gm([u for r in allres for u in r["ot"]["U"]]),
+            "stp": statistics.mean(u for r in allres for u in r["ot"]["STP"]),
+            "antt": statistics.mean(u for r in allres for u in r["ot"]["ANTT"]),
+            "mixes_per_s": world * args.steps / (omax / 1e3),
+            "throughput_speedup": nmax / omax,
+            "T_s_ms": dict(zip(tenants, np.mean(allres[0]["ot"]["ts_ms"], 0).tolist())),
+        }
         clocks = allres[0]["clk"]
         line = {
             "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": args.steps,
@@ -408,7 +430,7 @@ def main():
             "scaling": "weak", "vs_baseline": None, "dtype": "f32+i32", "data": "synthetic",
             "config": {"workload": CONFIGS.get(cfg_name, {}).get("desc", "config 5 mix per GPU"),
                        "config": cfg_name, "tenants": [r["tenants"] for r in allres] if world > 1 else tenants,
-                       "size": size, "mode": "SHARED (accelOS persistent, static quotas)",
+                       "size": size, "mode": f"SHARED (accelOS persistent CTAs, {args.policy} quotas)",
                        "l2": "flushed before every step (256 MiB write)",
                        "parallelism": f"independent mix per GPU x{world}"},
             "sharing": {
@@ -424,6 +446,8 @@ def main():
                 "T_s_ms_native": dict(zip(tenants, np.mean(na["ts_ms"], 0).tolist())),
                 "dispatch_overhead": {t: iso_persist[t] / iso_native[t] - 1 for t in tenants},
                 "native_mixes_per_s": world * args.steps / (nmax / 1e3),
+                "quotas_last_step": dict(zip(tenants, allres[0]["quotas"])),
+                "other_policy": other_sum,
             },
             "e2e": {"value": world * args.steps / (emax / 1e3), "unit": UNIT,
                     "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h},

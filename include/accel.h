@@ -97,6 +97,7 @@ typedef struct {
   const char *name;
   const void *persistent_fn;  /* host stub of accel_persistent<T>              */
   const void *native_fn;      /* host stub of accel_native<T>                  */
+  const void *topup_fn;       /* host stub of accel_topup<T> (RESOLVE growth)  */
   accel_dim3 block;           /* work-group (CTA) shape                        */
   uint32_t dyn_smem;          /* dynamic shared memory per CTA, bytes          */
   int32_t regs;               /* regs/thread for the solver; 0 = query attrs   */
@@ -200,6 +201,17 @@ int accel_stats(accel_ctx *ctx, uint64_t request_id, accel_req_stats *out);
  * ms_out[i] for launch i (steps in order, repeats in order), n = capacity;
  * *n_out = number of launches written. */
 int accel_launch_times(accel_ctx *ctx, uint64_t request_id, float *ms_out, uint32_t n, uint32_t *n_out);
+
+/* Per-launch device record of a completed request (from its Virtual NDRange
+ * descriptor): %globaltimer of the first CTA start / last CTA end, CTAs that
+ * got work, the admission high-water mark, the (dynamic) VG total, and whether
+ * a RESOLVE top-up joined.  out[n]; *n_out = launches written. */
+typedef struct {
+  uint64_t t_first_ns, t_last_ns;
+  uint32_t ctas_started, max_alive, total, topped;
+} accel_launch_stat;
+int accel_launch_stats(accel_ctx *ctx, uint64_t request_id, accel_launch_stat *out, uint32_t n,
+                       uint32_t *n_out);
 /* Forget completed requests (frees their descriptors); ACCEL_ALL = all done. */
 int accel_release(accel_ctx *ctx, uint64_t request_id);
 /* Streams of a tenant (cudaStream_t as void*), for interop (torch.cuda.ExternalStream). */

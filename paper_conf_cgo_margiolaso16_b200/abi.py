@@ -46,7 +46,8 @@ class accel_config(C.Structure):
 
 
 class accel_kernel_desc(C.Structure):
-    _fields_ = [("name", C.c_char_p), ("persistent_fn", vp), ("native_fn", vp), ("block", accel_dim3),
+    _fields_ = [("name", C.c_char_p), ("persistent_fn", vp), ("native_fn", vp), ("topup_fn", vp),
+                ("block", accel_dim3),
                 ("dyn_smem", u32), ("regs", i32), ("chunk", u32), ("args_size", u32)]
 
 
@@ -78,6 +79,11 @@ class accel_req_stats(C.Structure):
                 ("done_ms", f32), ("vgs_total", u32), ("launches", u32), ("quota_initial", u32),
                 ("quota_min", u32), ("quota_max", u32), ("resolves", u32), ("max_ctas", u32),
                 ("coverage_ok", i32), ("mode", i32)]
+
+
+class accel_launch_stat(C.Structure):
+    _fields_ = [("t_first_ns", u64), ("t_last_ns", u64), ("ctas_started", u32), ("max_alive", u32),
+                ("total", u32), ("topped", u32)]
 
 
 class accel_demand(C.Structure):
@@ -139,7 +145,7 @@ EXPORTS = [
     "accel_init", "accel_finalize", "accel_set_mode", "accel_last_error", "accel_builtin_kernel",
     "accel_builtin_count", "accel_builtin_name", "accel_kernel_register", "accel_kernel_info_get",
     "accel_submit", "accel_submit_group", "accel_sync", "accel_epoch", "accel_stats", "accel_release",
-    "accel_tenant_stream", "accel_launch_times", "accel_demand_of", "accel_solve", "accel_metrics", "accel_overlap",
+    "accel_tenant_stream", "accel_launch_times", "accel_launch_stats", "accel_demand_of", "accel_solve", "accel_metrics", "accel_overlap",
 ]
 
 
@@ -173,6 +179,7 @@ def _load() -> C.CDLL:
         "accel_release": (i32, [vp, u64]),
         "accel_tenant_stream": (i32, [vp, i32, P(vp), P(vp)]),
         "accel_launch_times": (i32, [vp, u64, P(f32), u32, P(u32)]),
+        "accel_launch_stats": (i32, [vp, u64, P(accel_launch_stat), u32, P(u32)]),
         "accel_demand_of": (i32, [P(accel_caps), u32, u32, u32, u32, u32, P(accel_demand)]),
         "accel_solve": (i32, [P(accel_caps), P(accel_demand), i32, P(u32)]),
         "accel_metrics": (i32, [P(f64), P(f64), i32, P(accel_mix_metrics)]),
@@ -263,6 +270,13 @@ def accel_launch_times(ctx, request_id: int, n: int) -> list[float]:
     buf = (f32 * max(n, 1))()
     got = u32()
     check(lib.accel_launch_times(ctx, request_id, buf, n, C.byref(got)), ctx)
+    return list(buf)[:got.value]
+
+
+def accel_launch_stats(ctx, request_id: int, n: int) -> list[accel_launch_stat]:
+    buf = (accel_launch_stat * max(n, 1))()
+    got = u32()
+    check(lib.accel_launch_stats(ctx, request_id, buf, n, C.byref(got)), ctx)
     return list(buf)[:got.value]
 
 

@@ -16,11 +16,24 @@
 //     static __device__ void body(const Args&, const VirtualBlock&, char* smem);
 // optionally  static constexpr bool kDynamicTotal = true;
 //             static __device__ uint32_t dynamic_total(const Args&, uint32_t launch_idx);
+//             static constexpr int kMinBlocks (same __launch_bounds__ both modes)
 // The body never reads blockIdx/gridDim (the `mop` test catches that), keeps
-// no state across VGs and never waits on another CTA, so the wrapper is
-// deadlock-free whatever the co-residency.
+// no state across VGs and never waits on another CTA.
 //   accel_persistent<T>: the reduced-grid scheduling kernel (Fig. 8b dyn_sched).
+//   accel_topup<T>:      RESOLVE growth grids (sticky across a step's launches).
 //   accel_native<T>:     the same body on the original grid (Fig. 1a baseline).
+//
+// RESOLVE policy (BASELINE.json north star; not in the paper, whose kernels
+// stay "bound to the resources initially allocated", lines 469-475): the
+// request's live quota lives in a device control word.  Admission is
+// count-based: a CTA works on a launch only while that launch's `alive` count
+// is <= live, so shrinking takes effect at the next dequeue of every CTA
+// (a VG boundary), and growing adds CTAs -- sticky top-up grids launched by the
+// host monitor on the tenant's second stream, which serve the current launch
+// and then follow the request's later launches.  Because a top-up CTA may
+// still run VGs of launch l after launch l's main grid retired, a launch whose
+// predecessor was topped up first waits for it to complete (queue exhausted
+// and no CTA alive) -- a wait on already-running CTAs only, so no deadlock.
 #pragma once
 
 #include <cstdint>
@@ -28,24 +41,33 @@
 
 namespace accel {
 
+// Per-request control block (device memory).
+struct Ctl {
+  uint32_t live;   // live quota (RESOLVE)
+  uint32_t cur;    // highest request-relative launch index started
+  uint32_t pad[2];
+};
+
 // Virtual NDRange of ONE launch ("Virtual Kernel Execution
-// Range which is copied to the accelerator memory").  128 B, two lines: the
-// read-mostly fields and stamps, then the hot dequeue counter on its own line.
+// Range which is copied to the accelerator memory").  256 B: read-mostly
+// fields and stamps, then the hot dequeue counter on its own 128-B line.
 struct alignas(128) Desc {
   uint32_t total;        // VGs in the original grid (static upper bound)
   uint32_t gx, gy, gz;   // original grid shape (decode, R-disp-2)
   uint32_t chunk;        // VGs per dequeue (§6.4)
   uint32_t launch_idx;   // index of this launch inside its step
   uint32_t flags;        // kFlag*
-  uint32_t total_seen;   // dynamic total as read by the CTAs (bfs)
-  uint32_t* live_quota;  // RESOLVE: CTAs with index >= *live_quota leave
+  uint32_t total_seen;   // total as read by the CTAs (dynamic for bfs)
+  Ctl* ctl;              // RESOLVE control block, nullptr otherwise
   uint32_t* coverage;    // verify: coverage[vg] += 1
   unsigned long long t_first;  // min %globaltimer over CTA starts
   unsigned long long t_last;   // max %globaltimer over CTA ends
-  uint32_t ctas_started; // CTAs that entered the scheduling loop
-  uint32_t alive;        // CTAs currently in the loop
+  uint32_t ctas_started; // CTAs admitted with work
+  uint32_t alive;        // CTAs currently admitted
   uint32_t max_alive;    // high-water mark of `alive`
-  uint32_t pad0[3];
+  uint32_t topped;       // a top-up CTA joined this launch
+  uint32_t req_idx;      // launch index inside the request
+  uint32_t has_prev;     // this - 1 is the request's previous launch
   // ---- line 1: the software queue head (RUN_TERMINATE when >= total)
   uint32_t next;
   uint32_t pad1[31];
@@ -120,52 +142,97 @@ __device__ __forceinline__ VirtualBlock decode(uint32_t vg, uint32_t gx, uint32_
 
 constexpr uint32_t kTerminate = 0xffffffffu;
 
-// One dequeue by the master thread (Fig. 8b line 26 rt_sched_wgroup):
-// RESOLVE shrink first (a CTA beyond the live quota leaves without consuming),
-// then one atomicAdd of `chunk` on the queue head.
-__device__ __forceinline__ uint32_t dequeue(Desc* d, uint32_t cta, uint32_t chunk) {
-  const uint32_t* lq = d->live_quota;
-  if (lq != nullptr && cta >= ld_volatile(lq)) return kTerminate;
+// A launch is complete when its queue is exhausted and no CTA is admitted
+// (a CTA is admitted before its first dequeue and leaves after its last VG).
+__device__ __forceinline__ void wait_complete(const Desc* p) {
+  for (;;) {
+    const uint32_t tot = ld_volatile(&p->total_seen);
+    if (tot != kTerminate && ld_volatile(&p->next) >= tot) {
+      __threadfence();
+      if (ld_volatile(&p->alive) == 0) break;
+    }
+    __nanosleep(256);
+  }
+  __threadfence();
+}
+
+// Master work-item, admission into launch d: count-based under RESOLVE,
+// plain alive tracking otherwise.  Returns false if the CTA must not work on d.
+__device__ __forceinline__ bool admit(Desc* d, uint32_t flags) {
+  const Ctl* ctl = d->ctl;
+  if (ctl != nullptr) {
+    const uint32_t a = atomicAdd(&d->alive, 1u) + 1u;
+    if (a > ld_volatile(&ctl->live)) {
+      atomicSub(&d->alive, 1u);
+      return false;
+    }
+    atomicMax(&d->max_alive, a);
+    __threadfence();  // admission visible before the first dequeue
+  } else if (flags & kFlagAlive) {
+    const uint32_t a = atomicAdd(&d->alive, 1u) + 1u;
+    atomicMax(&d->max_alive, a);
+  }
+  return true;
+}
+
+// One dequeue (Fig. 8b line 26, rt_sched_wgroup): under RESOLVE a CTA
+// leaves first if the launch holds more CTAs than the live quota (shrink at a
+// VG boundary); then one atomicAdd of `chunk` on the queue head.
+__device__ __forceinline__ uint32_t dequeue(Desc* d, uint32_t chunk, bool& admitted) {
+  const Ctl* ctl = d->ctl;
+  if (ctl != nullptr) {
+    const uint32_t live = ld_volatile(&ctl->live);
+    if (ld_volatile(&d->alive) > live) {
+      if (atomicSub(&d->alive, 1u) > live) {
+        admitted = false;
+        return kTerminate;
+      }
+      atomicAdd(&d->alive, 1u);
+    }
+  }
   return atomicAdd(&d->next, chunk);
 }
 
-// -------------------------------------------------------------------------
-// The scheduling kernel: grid = quota n_i (1-D), block = the original block.
-// cta_base > 0 for top-up launches that join a running Virtual NDRange.
+__device__ __forceinline__ void retire(Desc* d, uint32_t flags, bool admitted) {
+  if (admitted && (d->ctl != nullptr || (flags & kFlagAlive))) {
+    __threadfence();  // this CTA's VG results before the alive decrement
+    atomicSub(&d->alive, 1u);
+  }
+  if (flags & kFlagStamps) atomicMax(&d->t_last, globaltimer());
+}
+
+// Serve one launch: admission, dequeue loop, retire.  All threads call it.
 template <class T>
-__global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
-    accel_persistent(const typename T::Args args, Desc* __restrict__ d, uint32_t cta_base) {
-  extern __shared__ __align__(128) char smem[];
-  __shared__ uint32_t s_base[2];   // double-buffered dequeue result (sd.wg_base)
-  __shared__ uint32_t s_total;
-  const uint32_t cta = cta_base + blockIdx.x;
+__device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, char* smem,
+                                      uint32_t* s_base, uint32_t* s_total) {
   const uint32_t flags = d->flags;
   const uint32_t chunk = d->chunk;
   const uint32_t launch_idx = d->launch_idx;
   const uint32_t gx = d->gx, gy = d->gy, gz = d->gz;
   uint32_t* const coverage = d->coverage;
-
+  bool admitted = false;  // meaningful in thread 0 only
   if (threadIdx.x == 0) {  // master work-item: environment init (rt_env_init)
     if (flags & kFlagStamps) atomicMin(&d->t_first, globaltimer());
+    if (d->ctl != nullptr) atomicMax(&d->ctl->cur, d->req_idx);
     const uint32_t total = vg_total<T>(args, d, launch_idx);
-    s_total = total;
-    const uint32_t b = dequeue(d, cta, chunk);
-    s_base[0] = b;
-    if (b < total && (flags & kFlagAlive)) {
-      atomicAdd(&d->ctas_started, 1u);
-      const uint32_t a = atomicAdd(&d->alive, 1u) + 1u;
-      atomicMax(&d->max_alive, a);
+    *s_total = total;
+    if (d->total_seen != total) d->total_seen = total;
+    admitted = admit(d, flags);
+    uint32_t b = kTerminate;
+    if (admitted) {
+      b = dequeue(d, chunk, admitted);
+      if (b < total) atomicAdd(&d->ctas_started, 1u);
     }
+    s_base[0] = b;
   }
   __syncthreads();
-  const uint32_t total = s_total;
-  const bool started = s_base[0] < total;
+  const uint32_t total = *s_total;
   uint32_t buf = 0;
   for (;;) {
     const uint32_t base = s_base[buf];
     if (base >= total) break;                  // RUN_TERMINATE
     uint32_t nxt = 0;
-    if (threadIdx.x == 0) nxt = dequeue(d, cta, chunk);  // prefetch next chunk
+    if (threadIdx.x == 0) nxt = dequeue(d, chunk, admitted);  // prefetch next chunk
     const uint32_t end = min(base + chunk, total);
     for (uint32_t vg = base; vg < end; ++vg) {
       const VirtualBlock vb = decode(vg, gx, gy, gz, launch_idx);
@@ -177,10 +244,48 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
     __syncthreads();
     buf ^= 1;
   }
+  if (threadIdx.x == 0) retire(d, flags, admitted);
+}
+
+// -------------------------------------------------------------------------
+// The scheduling kernel: grid = quota (1-D), block = the original block;
+// serves launch d.
+template <class T>
+__global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
+    accel_persistent(const typename T::Args args, Desc* __restrict__ d, uint32_t /*unused*/) {
+  extern __shared__ __align__(128) char smem[];
+  __shared__ uint32_t s_base[2];   // double-buffered dequeue result (sd.wg_base)
+  __shared__ uint32_t s_total;
+  if (threadIdx.x == 0 && d->has_prev && ld_volatile(&(d - 1)->topped)) wait_complete(d - 1);
+  __syncthreads();
+  serve<T>(args, d, smem, s_base, &s_total);
+}
+
+// RESOLVE top-up grid: d = first launch of the request step, `sticky` =
+// launches in the step; starts at the request's current launch and follows
+// the step's later launches (each only once its predecessor completed).
+template <class T>
+__global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
+    accel_topup(const typename T::Args args, Desc* __restrict__ d, uint32_t sticky) {
+  extern __shared__ __align__(128) char smem[];
+  __shared__ uint32_t s_base[2];
+  __shared__ uint32_t s_total;
+  __shared__ uint32_t s_l;
   if (threadIdx.x == 0) {
-    if (started && (flags & kFlagAlive)) atomicSub(&d->alive, 1u);
-    if (flags & kFlagStamps) atomicMax(&d->t_last, globaltimer());
-    if (cta == 0) d->total_seen = total;
+    const uint32_t cur = ld_volatile(&d->ctl->cur);
+    s_l = cur > d->req_idx ? cur - d->req_idx : 0u;
+  }
+  __syncthreads();
+  for (uint32_t l = s_l; l < sticky; ++l) {
+    Desc* dl = d + l;
+    if (threadIdx.x == 0) {
+      if (dl->has_prev) wait_complete(dl - 1);  // launch l's inputs are complete
+      atomicExch(&dl->topped, 1u);
+      __threadfence();
+    }
+    __syncthreads();
+    serve<T>(args, dl, smem, s_base, &s_total);
+    __syncthreads();
   }
 }
 

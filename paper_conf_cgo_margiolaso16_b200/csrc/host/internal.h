@@ -9,6 +9,7 @@
 namespace accel {
 
 struct Desc;  // csrc/device/dispatch.cuh
+struct Ctl;
 
 struct InitStep {
   uint32_t first;      // first descriptor of the step
@@ -21,7 +22,7 @@ struct InitStep {
 
 struct InitParams {
   Desc* d;
-  uint32_t* live_quota;   // nullptr under STATIC
+  Ctl* ctl;               // RESOLVE control block, nullptr under STATIC
   uint32_t live_init;     // initial live quota of the main step
   uint32_t* coverage;     // nullptr unless verify
   uint32_t flags;
@@ -31,6 +32,9 @@ struct InitParams {
 
 // Fill the descriptors of one request on `s` (one tiny kernel).
 cudaError_t launch_desc_init(const InitParams& p, uint32_t n_desc, cudaStream_t s);
+// RESOLVE: wait (1 thread) until the request's last launch and its top-ups completed.
+cudaError_t launch_join(const Desc* last, cudaStream_t s);
 constexpr size_t kDescBytes = 256;
+constexpr size_t kCtlBytes = 16;
 
 }  // namespace accel

@@ -12,12 +12,16 @@
 #include <cuda_runtime.h>
 
 #include <algorithm>
+#include <atomic>
+#include <chrono>
 #include <cstdio>
+#include <cstdlib>
 #include <cstring>
 #include <map>
 #include <memory>
 #include <mutex>
 #include <string>
+#include <thread>
 #include <vector>
 
 #include "accel.h"
@@ -26,6 +30,7 @@
 namespace {
 
 using accel::InitParams;
+using accel::kCtlBytes;
 using accel::kDescBytes;
 
 constexpr uint32_t kPoolSlots = 16384;      // 4 MiB of descriptors
@@ -35,6 +40,7 @@ struct Kernel {
   std::string name;
   const void* pfn;
   const void* nfn;
+  const void* tfn;
   dim3 block;
   uint32_t dyn_smem;
   uint32_t chunk;
@@ -72,7 +78,10 @@ struct Request {
   uint32_t* cov = nullptr;
   uint64_t cov_elems = 0;
   uint32_t quota_initial = 0, quota_min = 0, quota_max = 0, resolves = 0;
+  uint32_t live = 0;         // RESOLVE: current live quota of the main step
+  uint32_t provisioned = 0;  // RESOLVE: main-grid CTAs + sticky top-up CTAs
   bool done = false;
+  bool departed_seen = false;  // monitor already re-solved for this departure
   bool fetched = false;
   int cov_ok = -1;
   std::vector<unsigned char> desc_host;
@@ -103,7 +112,7 @@ struct DescHost {
   uint32_t total, gx, gy, gz, chunk, launch_idx, flags, total_seen;
   uint64_t live_quota, coverage;
   unsigned long long t_first, t_last;
-  uint32_t ctas_started, alive, max_alive;
+  uint32_t ctas_started, alive, max_alive, topped, req_idx, has_prev;
 };
 
 }  // namespace
@@ -116,12 +125,22 @@ struct accel_ctx {
   bool poisoned = false;
   std::vector<Kernel> kernels;
   cudaStream_t main[ACCEL_MAX_TENANTS] = {};
-  cudaStream_t topup[ACCEL_MAX_TENANTS] = {};
+  // RESOLVE top-up grids are sticky (they follow a request's launches), so two
+  // of them must never share a stream: a pool with its own hardware queues
+  // (16 main + 12 top-up + 1 control <= CUDA_DEVICE_MAX_CONNECTIONS = 32).
+  static constexpr int kTopupStreams = 12;
+  cudaStream_t topup[kTopupStreams] = {};
+  uint32_t topup_rr = 0;
   cudaStream_t ctl = nullptr;
   cudaEvent_t epoch = nullptr;
   bool epoch_set = false;
   unsigned char* pool = nullptr;
-  uint32_t* quota_words = nullptr;
+  unsigned char* ctl_pool = nullptr;      // accel::Ctl per descriptor slot
+  uint32_t* pinned_ring = nullptr;        // staging for live-quota writes
+  uint32_t ring_pos = 0;
+  std::thread monitor;
+  std::atomic<bool> stop{false};
+  uint64_t monitor_solves = 0;
   std::vector<uint8_t> slot_used;
   std::map<uint64_t, std::unique_ptr<Request>> reqs;
   uint64_t next_id = 1;
@@ -160,6 +179,7 @@ struct accel_ctx {
   }
   void free_slots(uint32_t s, uint32_t n) { std::fill(slot_used.begin() + s, slot_used.begin() + s + n, 0); }
   accel::Desc* desc_ptr(uint32_t slot) { return reinterpret_cast<accel::Desc*>(pool + (size_t)slot * kDescBytes); }
+  accel::Ctl* ctl_ptr(uint32_t slot) { return reinterpret_cast<accel::Ctl*>(ctl_pool + (size_t)slot * kCtlBytes); }
 };
 
 #define CK(ctx, call)                                  \
@@ -235,7 +255,7 @@ int enqueue(accel_ctx* ctx, Request* r) {
   InitParams p{};
   p.d = ctx->desc_ptr(r->slot);
   const bool resolve = shared && ctx->cfg.policy == ACCEL_POLICY_RESOLVE;
-  p.live_quota = resolve ? ctx->quota_words + r->slot : nullptr;
+  p.ctl = resolve ? ctx->ctl_ptr(r->slot) : nullptr;
   p.live_init = r->steps[r->main_step].quota;
   p.coverage = r->cov;
   p.flags = kFlagStamps | (shared ? kFlagAlive : 0u);
@@ -258,13 +278,14 @@ int enqueue(accel_ctx* ctx, Request* r) {
     for (uint32_t l = 0; l < st.repeat; ++l, ++li) {
       if (lev) CK(ctx, cudaEventRecord(r->ev_launch[li], s));
       accel::Desc* d = ctx->desc_ptr(r->slot + st.first + l);
-      uint32_t cta_base = 0;
-      void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &cta_base};
+      uint32_t sticky = 0;
+      void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &sticky};
       const dim3 grid = shared ? dim3(st.quota, 1, 1) : dim3(st.grid.x, st.grid.y, st.grid.z);
       CK(ctx, cudaLaunchKernel(shared ? k.pfn : k.nfn, grid, k.block, params, k.dyn_smem, s));
     }
   }
   if (lev) CK(ctx, cudaEventRecord(r->ev_launch[li], s));
+  if (resolve) CK(ctx, accel::launch_join(ctx->desc_ptr(r->slot + r->n_desc - 1), s));
   for (const accel_copy& c : r->d2h) CK(ctx, cudaMemcpyAsync(c.dst, c.src, c.bytes, cudaMemcpyDeviceToHost, s));
   CK(ctx, cudaEventRecord(r->ev_done, s));
   return ACCEL_OK;
@@ -315,8 +336,43 @@ int build_request(accel_ctx* ctx, const accel_request& in, std::unique_ptr<Reque
   return ACCEL_OK;
 }
 
-// Solve over active requests (arrival order) + the new ones; assign the new
-// ones' quotas (STATIC: running requests keep theirs).
+constexpr uint32_t kRing = 4096;
+
+// RESOLVE: set a running request's live quota (copy engine, no SM needed) and
+// add sticky top-up CTAs when it grows beyond what is provisioned.
+bool debug_on() {
+  static const bool on = std::getenv("ACCEL_DEBUG") != nullptr;
+  return on;
+}
+
+int apply_quota(accel_ctx* ctx, Request* r, uint32_t q) {
+  if (debug_on())
+    std::fprintf(stderr, "[accel] resolve req %llu tenant %d live %u -> %u (provisioned %u)\n",
+                 (unsigned long long)r->id, r->tenant, r->live, q, r->provisioned);
+  if (q == r->live) return ACCEL_OK;
+  uint32_t* h = ctx->pinned_ring + (ctx->ring_pos++ % kRing);
+  *h = q;
+  CK(ctx, cudaMemcpyAsync(ctx->ctl_pool + (size_t)r->slot * kCtlBytes /* Ctl::live */, h, sizeof(uint32_t), cudaMemcpyHostToDevice, ctx->ctl));
+  if (q > r->provisioned) {
+    const Step& st = r->steps[r->main_step];
+    const Kernel& k = ctx->kernels[st.kid];
+    accel::Desc* d = ctx->desc_ptr(r->slot + st.first);
+    uint32_t sticky = st.repeat;
+    void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &sticky};
+    CK(ctx, cudaLaunchKernel(k.tfn, dim3(q - r->provisioned, 1, 1), k.block, params, k.dyn_smem,
+                             ctx->topup[ctx->topup_rr++ % accel_ctx::kTopupStreams]));
+    r->provisioned = q;
+  }
+  r->live = q;
+  r->resolves += 1;
+  r->quota_min = std::min(r->quota_min, q);
+  r->quota_max = std::max(r->quota_max, q);
+  return ACCEL_OK;
+}
+
+// Solve over the active requests (arrival order) + the new ones.  STATIC:
+// running requests keep their quota and only the new
+// ones are assigned.  RESOLVE: every active request gets its new quota.
 int assign_quotas(accel_ctx* ctx, std::vector<std::unique_ptr<Request>>& fresh) {
   std::vector<Request*> order;
   for (auto& kv : ctx->reqs) {
@@ -326,6 +382,7 @@ int assign_quotas(accel_ctx* ctx, std::vector<std::unique_ptr<Request>>& fresh) 
     if (!r->done && r->mode == ACCEL_MODE_SHARED) order.push_back(r);
   }
   for (auto& r : fresh) order.push_back(r.get());
+  if (order.empty()) return ACCEL_OK;
   std::vector<accel_demand> ds(order.size());
   for (size_t i = 0; i < order.size(); ++i) {
     Request* r = order[i];
@@ -335,7 +392,13 @@ int assign_quotas(accel_ctx* ctx, std::vector<std::unique_ptr<Request>>& fresh) 
   std::vector<uint32_t> q(order.size());
   int rc = accel_solve(&ctx->caps, ds.data(), (int32_t)ds.size(), q.data());
   if (rc) return ctx->fail(rc, "accel_solve failed");
+  ctx->monitor_solves += 1;
   const size_t first_new = order.size() - fresh.size();
+  if (ctx->cfg.policy == ACCEL_POLICY_RESOLVE)
+    for (size_t i = 0; i < first_new; ++i) {
+      rc = apply_quota(ctx, order[i], q[i]);
+      if (rc) return rc;
+    }
   for (size_t i = first_new; i < order.size(); ++i) {
     Request* r = order[i];
     for (size_t j = 0; j < r->steps.size(); ++j) {
@@ -350,8 +413,41 @@ int assign_quotas(accel_ctx* ctx, std::vector<std::unique_ptr<Request>>& fresh) 
       }
     }
     r->quota_initial = r->quota_min = r->quota_max = q[i];
+    r->live = r->provisioned = q[i];
   }
   return ACCEL_OK;
+}
+
+// Host monitor (RESOLVE): detects departures without host synchronisation by
+// polling the requests' completion events, and re-solves the survivors.
+void monitor_loop(accel_ctx* ctx) {
+  cudaSetDevice(ctx->cfg.device);
+  bool busy = false;
+  while (!ctx->stop.load()) {
+    std::this_thread::sleep_for(std::chrono::microseconds(busy ? 20 : 500));
+    std::unique_lock<std::mutex> g(ctx->mu);
+    busy = false;
+    if (ctx->poisoned || ctx->cfg.mode != ACCEL_MODE_SHARED || ctx->cfg.policy != ACCEL_POLICY_RESOLVE)
+      continue;
+    bool departed = false, running = false;
+    for (auto& kv : ctx->reqs) {
+      Request* r = kv.second.get();
+      if (r->mode != ACCEL_MODE_SHARED || r->departed_seen) continue;
+      if (refresh_done(ctx, r)) break;
+      if (r->done) {
+        r->departed_seen = true;
+        departed = true;
+      } else {
+        running = true;
+      }
+    }
+    busy = running;
+    if (departed && debug_on()) std::fprintf(stderr, "[accel] monitor: departure (running=%d)\n", (int)running);
+    if (departed && running) {
+      std::vector<std::unique_ptr<Request>> none;
+      assign_quotas(ctx, none);
+    }
+  }
 }
 
 int submit_locked(accel_ctx* ctx, uint32_t n, const accel_request* rs, uint64_t* ids) {
@@ -423,26 +519,33 @@ int accel_init(const accel_config* cfg, accel_ctx** out) {
   if (e != cudaSuccess) return init_fail(e, "cudaDeviceGetAttribute");
   ctx->caps = cfg->caps;
   if (ctx->caps.sms <= 0) ctx->caps.sms = sms;
-  for (int t = 0; t < ACCEL_MAX_TENANTS; ++t) {
+  for (int t = 0; t < ACCEL_MAX_TENANTS; ++t)
     if ((e = cudaStreamCreateWithFlags(&ctx->main[t], cudaStreamNonBlocking)) != cudaSuccess)
       return init_fail(e, "cudaStreamCreate");
+  for (int t = 0; t < accel_ctx::kTopupStreams; ++t)
     if ((e = cudaStreamCreateWithFlags(&ctx->topup[t], cudaStreamNonBlocking)) != cudaSuccess)
       return init_fail(e, "cudaStreamCreate");
-  }
   if ((e = cudaStreamCreateWithFlags(&ctx->ctl, cudaStreamNonBlocking)) != cudaSuccess)
     return init_fail(e, "cudaStreamCreate");
   if ((e = cudaEventCreate(&ctx->epoch)) != cudaSuccess) return init_fail(e, "cudaEventCreate");
   if ((e = cudaMalloc(&ctx->pool, (size_t)kPoolSlots * kDescBytes)) != cudaSuccess)
     return init_fail(e, "cudaMalloc(pool)");
-  if ((e = cudaMalloc(&ctx->quota_words, (size_t)kPoolSlots * sizeof(uint32_t))) != cudaSuccess)
-    return init_fail(e, "cudaMalloc(quota)");
+  if ((e = cudaMalloc(&ctx->ctl_pool, (size_t)kPoolSlots * kCtlBytes)) != cudaSuccess)
+    return init_fail(e, "cudaMalloc(ctl)");
+  if ((e = cudaHostAlloc(reinterpret_cast<void**>(&ctx->pinned_ring), kRing * sizeof(uint32_t),
+                         cudaHostAllocDefault)) != cudaSuccess)
+    return init_fail(e, "cudaHostAlloc(ring)");
   ctx->slot_used.assign(kPoolSlots, 0);
-  *out = ctx.release();
+  accel_ctx* raw = ctx.release();
+  raw->monitor = std::thread(monitor_loop, raw);
+  *out = raw;
   return ACCEL_OK;
 }
 
 int accel_finalize(accel_ctx* ctx) {
   if (!ctx) return ACCEL_OK;
+  ctx->stop.store(true);
+  if (ctx->monitor.joinable()) ctx->monitor.join();
   cudaSetDevice(ctx->cfg.device);
   for (auto& kv : ctx->reqs) {
     if (kv.second->ev_done) cudaEventSynchronize(kv.second->ev_done);
@@ -450,14 +553,15 @@ int accel_finalize(accel_ctx* ctx) {
   }
   ctx->reqs.clear();
   for (cudaEvent_t ev : ctx->free_events) cudaEventDestroy(ev);
-  for (int t = 0; t < ACCEL_MAX_TENANTS; ++t) {
+  for (int t = 0; t < ACCEL_MAX_TENANTS; ++t)
     if (ctx->main[t]) cudaStreamDestroy(ctx->main[t]);
+  for (int t = 0; t < accel_ctx::kTopupStreams; ++t)
     if (ctx->topup[t]) cudaStreamDestroy(ctx->topup[t]);
-  }
   if (ctx->ctl) cudaStreamDestroy(ctx->ctl);
   if (ctx->epoch) cudaEventDestroy(ctx->epoch);
   if (ctx->pool) cudaFree(ctx->pool);
-  if (ctx->quota_words) cudaFree(ctx->quota_words);
+  if (ctx->ctl_pool) cudaFree(ctx->ctl_pool);
+  if (ctx->pinned_ring) cudaFreeHost(ctx->pinned_ring);
   delete ctx;
   return ACCEL_OK;
 }
@@ -487,6 +591,7 @@ int accel_kernel_register(accel_ctx* ctx, const accel_kernel_desc* d, int32_t* k
   k.name = d->name ? d->name : "?";
   k.pfn = d->persistent_fn;
   k.nfn = d->native_fn;
+  k.tfn = d->topup_fn ? d->topup_fn : d->persistent_fn;
   k.block = dim3(d->block.x, d->block.y ? d->block.y : 1, d->block.z ? d->block.z : 1);
   k.dyn_smem = d->dyn_smem;
   k.chunk = d->chunk ? d->chunk : 1;
@@ -496,7 +601,7 @@ int accel_kernel_register(accel_ctx* ctx, const accel_kernel_desc* d, int32_t* k
   if ((int)k.threads() > a.maxThreadsPerBlock) return ctx->fail(ACCEL_ENOFIT, "block larger than the kernel allows");
   k.num_regs = d->regs > 0 ? d->regs : a.numRegs;
   k.static_smem = (int)a.sharedSizeBytes;
-  for (const void* fn : {k.pfn, k.nfn}) {
+  for (const void* fn : {k.pfn, k.nfn, k.tfn}) {
     if (k.dyn_smem > 48 * 1024)
       CK(ctx, cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)k.dyn_smem));
     // one carveout for every tenant so CTAs of different kernels can share an SM
@@ -545,25 +650,34 @@ int accel_submit(accel_ctx* ctx, const accel_request* r, uint64_t* id) {
 
 int accel_sync(accel_ctx* ctx, uint64_t request_id) {
   if (!ctx) return ACCEL_EINVAL;
-  std::lock_guard<std::mutex> g(ctx->mu);
-  if (ctx->poisoned) return ACCEL_ESTATE;
-  CK(ctx, cudaSetDevice(ctx->cfg.device));
-  std::vector<Request*> todo;
-  if (request_id == ACCEL_ALL) {
-    for (auto& kv : ctx->reqs) todo.push_back(kv.second.get());
-  } else {
-    auto it = ctx->reqs.find(request_id);
-    if (it == ctx->reqs.end()) return ctx->fail(ACCEL_EINVAL, "unknown request");
-    todo.push_back(it->second.get());
-  }
-  for (Request* r : todo) {
-    if (!r->done) {
-      CK(ctx, cudaEventSynchronize(r->ev_done));
-      r->done = true;
+  std::vector<std::pair<uint64_t, cudaEvent_t>> wait;
+  {
+    std::lock_guard<std::mutex> g(ctx->mu);
+    if (ctx->poisoned) return ACCEL_ESTATE;
+    CK(ctx, cudaSetDevice(ctx->cfg.device));
+    if (request_id == ACCEL_ALL) {
+      for (auto& kv : ctx->reqs) wait.emplace_back(kv.first, kv.second->ev_done);
+    } else {
+      auto it = ctx->reqs.find(request_id);
+      if (it == ctx->reqs.end()) return ctx->fail(ACCEL_EINVAL, "unknown request");
+      wait.emplace_back(request_id, it->second->ev_done);
     }
   }
+  // wait without the lock: the RESOLVE monitor keeps re-solving meanwhile
+  for (auto& w : wait) {
+    cudaError_t e = cudaEventSynchronize(w.second);
+    if (e != cudaSuccess) {
+      std::lock_guard<std::mutex> g(ctx->mu);
+      return ctx->cuda(e, "cudaEventSynchronize");
+    }
+  }
+  std::lock_guard<std::mutex> g(ctx->mu);
   bool cov_bad = false;
-  for (Request* r : todo) {
+  for (auto& w : wait) {
+    auto it = ctx->reqs.find(w.first);
+    if (it == ctx->reqs.end()) continue;
+    Request* r = it->second.get();
+    r->done = true;
     int rc = fetch_result(ctx, r);
     if (rc) return rc;
     if (r->cov_ok == 0) cov_bad = true;
@@ -642,6 +756,33 @@ int accel_launch_times(accel_ctx* ctx, uint64_t request_id, float* ms_out, uint3
   return ACCEL_OK;
 }
 
+int accel_launch_stats(accel_ctx* ctx, uint64_t request_id, accel_launch_stat* out, uint32_t n,
+                       uint32_t* n_out) {
+  if (!ctx || (n && !out) || !n_out) return ACCEL_EINVAL;
+  std::lock_guard<std::mutex> g(ctx->mu);
+  if (ctx->poisoned) return ACCEL_ESTATE;
+  auto it = ctx->reqs.find(request_id);
+  if (it == ctx->reqs.end()) return ctx->fail(ACCEL_EINVAL, "unknown request");
+  Request* r = it->second.get();
+  int rc = refresh_done(ctx, r);
+  if (rc) return rc;
+  if (!r->done) return ACCEL_ENOTREADY;
+  rc = fetch_result(ctx, r);
+  if (rc) return rc;
+  const uint32_t m = std::min<uint32_t>(n, r->n_desc);
+  for (uint32_t i = 0; i < m; ++i) {
+    const DescHost* d = reinterpret_cast<const DescHost*>(r->desc_host.data() + (size_t)i * kDescBytes);
+    out[i].t_first_ns = d->t_first;
+    out[i].t_last_ns = d->t_last;
+    out[i].ctas_started = d->ctas_started;
+    out[i].max_alive = d->max_alive;
+    out[i].total = d->total_seen;
+    out[i].topped = d->topped;
+  }
+  *n_out = m;
+  return ACCEL_OK;
+}
+
 int accel_release(accel_ctx* ctx, uint64_t request_id) {
   if (!ctx) return ACCEL_EINVAL;
   std::lock_guard<std::mutex> g(ctx->mu);
@@ -667,7 +808,7 @@ int accel_release(accel_ctx* ctx, uint64_t request_id) {
 int accel_tenant_stream(accel_ctx* ctx, int32_t tenant, void** main_stream, void** topup_stream) {
   if (!ctx || tenant < 0 || tenant >= ACCEL_MAX_TENANTS) return ACCEL_EINVAL;
   if (main_stream) *main_stream = ctx->main[tenant];
-  if (topup_stream) *topup_stream = ctx->topup[tenant];
+  if (topup_stream) *topup_stream = ctx->topup[tenant % accel_ctx::kTopupStreams];
   return ACCEL_OK;
 }
 

@@ -7,17 +7,24 @@
 
 #include "device/dispatch.cuh"
 #include "host/internal.h"
+#include "tenants/bfs.cuh"
+#include "tenants/cutcp.cuh"
 #include "tenants/histo.cuh"
 #include "tenants/mop.cuh"
 #include "tenants/stencil.cuh"
+#include "tenants/tpacf.cuh"
 
 namespace accel {
 
 static_assert(sizeof(Desc) == kDescBytes, "descriptor size");
+static_assert(sizeof(Ctl) == kCtlBytes, "control block size");
 
 __global__ void desc_init_kernel(const InitParams p, uint32_t n_desc) {
   const uint32_t i = blockIdx.x * blockDim.x + threadIdx.x;
-  if (i == 0 && p.live_quota != nullptr) *p.live_quota = p.live_init;
+  if (i == 0 && p.ctl != nullptr) {
+    p.ctl->live = p.live_init;
+    p.ctl->cur = 0;
+  }
   if (i >= n_desc) return;
   uint32_t s = 0;
   while (s + 1 < p.n_steps && i >= p.steps[s + 1].first) ++s;
@@ -31,15 +38,27 @@ __global__ void desc_init_kernel(const InitParams p, uint32_t n_desc) {
   d->chunk = st.chunk;
   d->launch_idx = r;
   d->flags = p.flags;
-  d->total_seen = 0xffffffffu;
-  d->live_quota = p.live_quota;
+  d->total_seen = kTerminate;
+  d->ctl = p.ctl;
   d->coverage = p.coverage ? p.coverage + st.cov_offset + (size_t)r * st.total : nullptr;
   d->t_first = ULLONG_MAX;
   d->t_last = 0;
   d->ctas_started = 0;
   d->alive = 0;
   d->max_alive = 0;
+  d->topped = 0;
+  d->req_idx = i;
+  d->has_prev = i > 0 ? 1u : 0u;
   d->next = 0;
+}
+
+__global__ void join_kernel(const Desc* last) {
+  if (threadIdx.x == 0 && ld_volatile(&last->topped)) wait_complete(last);
+}
+
+cudaError_t launch_join(const Desc* last, cudaStream_t s) {
+  join_kernel<<<1, 32, 0, s>>>(last);
+  return cudaGetLastError();
 }
 
 cudaError_t launch_desc_init(const InitParams& p, uint32_t n_desc, cudaStream_t s) {
@@ -55,6 +74,7 @@ accel_kernel_desc make_desc(const char* name) {
   d.name = name;
   d.persistent_fn = reinterpret_cast<const void*>(&accel_persistent<T>);
   d.native_fn = reinterpret_cast<const void*>(&accel_native<T>);
+  d.topup_fn = reinterpret_cast<const void*>(&accel_topup<T>);
   d.block = accel_dim3{(uint32_t)T::kThreads, 1u, 1u};
   d.dyn_smem = T::kDynSmem;
   d.regs = 0;
@@ -72,6 +92,9 @@ const Builtin kBuiltins[] = {
     {"mop", &make_desc<Mop>},
     {"stencil", &make_desc<Stencil>},
     {"histo", &make_desc<Histo>},
+    {"bfs", &make_desc<Bfs>},
+    {"cutcp", &make_desc<Cutcp>},
+    {"tpacf", &make_desc<Tpacf>},
 };
 constexpr int kNumBuiltins = sizeof(kBuiltins) / sizeof(kBuiltins[0]);
 }  // namespace

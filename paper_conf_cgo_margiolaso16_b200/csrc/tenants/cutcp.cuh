@@ -1,0 +1,108 @@
+// cutcp -- cutoff Coulombic potential on a 3-D lattice (Parboil "cutcp",
+// PAPER.md lines 290-291, 978).
+//
+// One VG = 8 x 8 x 8 lattice points; 128 threads, thread t owns the column
+// (i, j) = (t % 8, (t / 8) % 8) and 4 consecutive k.  Atoms arrive binned in
+// cells (x fastest); a row of cells along x is one contiguous atom range, so
+// the VG walks the (y, z) cell rows whose distance to the VG box is < cutoff,
+// trims each row's x-range to the sphere, stages the atoms in shared memory
+// (128 float4 per tile) and every thread tests them against its 4 points.
+// Membership r^2 < c^2 and the exclusion r^2 < e^2 are decided on the fp32
+// value ((dx*dx + dy*dy) + dz*dz, round-to-nearest, no FMA) exactly like the
+// oracle (DESIGN.md R-fp-1); the term q/r (1 - r^2/c^2)^2 is fp32.
+// FP32-ALU bound (+ MUFU rsqrt for in-range pairs).
+#pragma once
+#include "../device/dispatch.cuh"
+#include "accel_tenants.h"
+
+namespace accel {
+
+struct Cutcp {
+  using Args = accel_cutcp_args;
+  static constexpr int kThreads = 128;
+  static constexpr uint32_t kChunk = 1;
+  static constexpr int kMinBlocks = 8;
+  static constexpr int kTile = 128;  // atoms staged per round
+  static constexpr int kPts = 4;     // points per thread along z
+  static constexpr uint32_t kDynSmem = kTile * sizeof(float4);
+
+  static __device__ __forceinline__ float gap(float lo, float hi, float clo, float chi) {
+    // distance between intervals [lo, hi] and [clo, chi]
+    return fmaxf(0.f, fmaxf(clo - hi, lo - chi));
+  }
+
+  static __device__ __forceinline__ void body(const Args& a, const VirtualBlock& vb, char* smem) {
+    float4* tile = reinterpret_cast<float4*>(smem);
+    const int t = threadIdx.x;
+    const int i = vb.x * 8 + (t & 7);
+    const int j = vb.y * 8 + ((t >> 3) & 7);
+    const int k0 = vb.z * 8 + (t >> 6) * kPts;
+    const float h = a.h;
+    const float px = h * (float)i, py = h * (float)j;
+    float pz[kPts];
+#pragma unroll
+    for (int p = 0; p < kPts; ++p) pz[p] = h * (float)(k0 + p);
+    const float c = a.cutoff;
+    const float c2 = c * c, e2 = a.excl * a.excl, inv_c2 = 1.0f / c2;
+    float sum[kPts];
+    bool excl[kPts];
+#pragma unroll
+    for (int p = 0; p < kPts; ++p) {
+      sum[p] = 0.f;
+      excl[p] = false;
+    }
+    // VG bounding box in Angstrom
+    const float bx0 = h * (float)(vb.x * 8), bx1 = h * (float)(vb.x * 8 + 7);
+    const float by0 = h * (float)(vb.y * 8), by1 = h * (float)(vb.y * 8 + 7);
+    const float bz0 = h * (float)(vb.z * 8), bz1 = h * (float)(vb.z * 8 + 7);
+    const float cs = a.cell;
+    const int nc = (int)a.ncell;
+    const float cm = c + 0.05f;  // conservative margin for the cell filter
+    auto clampc = [&](int v) { return v < 0 ? 0 : (v >= nc ? nc - 1 : v); };
+    const int cy0 = clampc((int)floorf((by0 - cm) / cs)), cy1 = clampc((int)floorf((by1 + cm) / cs));
+    const int cz0 = clampc((int)floorf((bz0 - cm) / cs)), cz1 = clampc((int)floorf((bz1 + cm) / cs));
+    for (int cz = cz0; cz <= cz1; ++cz) {
+      const float gz = gap(bz0, bz1, cz * cs, (cz + 1) * cs);
+      for (int cy = cy0; cy <= cy1; ++cy) {
+        const float gy = gap(by0, by1, cy * cs, (cy + 1) * cs);
+        const float d2 = gy * gy + gz * gz;
+        if (d2 >= cm * cm) continue;  // uniform across the CTA
+        const float rx = sqrtf(cm * cm - d2);
+        const int cx0 = clampc((int)floorf((bx0 - rx) / cs)), cx1 = clampc((int)floorf((bx1 + rx) / cs));
+        const int row = (cz * nc + cy) * nc;
+        const int a0 = __ldg(a.cell_start + row + cx0), a1 = __ldg(a.cell_start + row + cx1 + 1);
+        for (int base = a0; base < a1; base += kTile) {
+          const int n = min(kTile, a1 - base);
+          __syncthreads();
+          if (t < n) tile[t] = __ldg(reinterpret_cast<const float4*>(a.atoms) + base + t);
+          __syncthreads();
+#pragma unroll 2
+          for (int q = 0; q < n; ++q) {
+            const float4 at = tile[q];
+            const float dx = __fsub_rn(px, at.x), dy = __fsub_rn(py, at.y);
+            const float dxy = __fadd_rn(__fmul_rn(dx, dx), __fmul_rn(dy, dy));
+#pragma unroll
+            for (int p = 0; p < kPts; ++p) {
+              const float dz = __fsub_rn(pz[p], at.z);
+              const float r2 = __fadd_rn(dxy, __fmul_rn(dz, dz));
+              excl[p] |= r2 < e2;
+              if (r2 < c2) {
+                const float s = 1.0f - r2 * inv_c2;
+                sum[p] += at.w * rsqrtf(r2) * s * s;
+              }
+            }
+          }
+        }
+      }
+    }
+    if (i < (int)a.nx && j < (int)a.ny) {
+#pragma unroll
+      for (int p = 0; p < kPts; ++p) {
+        const int k = k0 + p;
+        if (k < (int)a.nz) a.v[((size_t)k * a.ny + j) * a.nx + i] = excl[p] ? 0.f : sum[p];
+      }
+    }
+  }
+};
+
+}  // namespace accel

@@ -47,8 +47,22 @@ struct Histo {
     const uint64_t per_vec = 16 / sb;
     const uint64_t nvec = (hi - lo) / per_vec;
     const uint4* v = reinterpret_cast<const uint4*>(base + lo * sb);
-    for (uint64_t i = threadIdx.x; i < nvec; i += kThreads) {
-      const uint4 w = __ldcs(v + i);   // streamed once: evict-first
+    // four independent 16-B loads in flight per thread before counting
+    uint64_t i = threadIdx.x;
+    for (; i + 3 * kThreads < nvec; i += 4 * kThreads) {
+      uint4 w[4];
+#pragma unroll
+      for (int u = 0; u < 4; ++u) w[u] = __ldcs(v + i + u * kThreads);  // streamed once
+#pragma unroll
+      for (int u = 0; u < 4; ++u) {
+        count4(h, w[u].x, sb);
+        count4(h, w[u].y, sb);
+        count4(h, w[u].z, sb);
+        count4(h, w[u].w, sb);
+      }
+    }
+    for (; i < nvec; i += kThreads) {
+      const uint4 w = __ldcs(v + i);
       count4(h, w.x, sb);
       count4(h, w.y, sb);
       count4(h, w.z, sb);

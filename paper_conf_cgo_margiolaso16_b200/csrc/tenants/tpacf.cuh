@@ -1,0 +1,100 @@
+// tpacf -- two-point angular correlation histograms (Parboil "tpacf",
+// PAPER.md lines 290-298, 1132).
+//
+// VG (x, y): 256 points i of block x from set P against every point j of set
+// Q; y = 0 -> DD (P = Q = data, pairs i < j), y = 1..S -> RR of random set
+// y-1 (i < j), y = S+1..2S -> DR (data x random set y-S-1, all pairs).  Q is
+// staged through shared memory in tiles of 256 points (broadcast reads).  The
+// angular bin of a pair is decided on the fp32 dot product
+// (x*x' + y*y') + z*z' (round-to-nearest, no FMA, DESIGN.md R-fp-1) by a
+// binary search over the descending bin edges; each lane counts into its own
+// shared-memory sub-histogram column (conflict-free, no atomics); the VG ends
+// with one 64-bit global atomic per bin.  Integer result: bit-exact.
+#pragma once
+#include "../device/dispatch.cuh"
+#include "accel_tenants.h"
+
+namespace accel {
+
+struct Tpacf {
+  using Args = accel_tpacf_args;
+  static constexpr int kThreads = 256;
+  static constexpr uint32_t kChunk = 1;
+  static constexpr int kMinBlocks = 6;   // <= 40 regs: smem allows 6 CTAs/SM
+  static constexpr int kWarps = kThreads / 32;
+  static constexpr int kMaxBins = 32;      // nedges + 1 <= 32
+  static constexpr int kTile = 256;
+  // [warp][bin][lane] u32 counters + Q tile (3 x 256 floats) + edges (32)
+  static constexpr uint32_t kDynSmem =
+      kWarps * kMaxBins * 32 * sizeof(uint32_t) + 3 * kTile * sizeof(float) + 32 * sizeof(float);
+
+  static __device__ __forceinline__ void body(const Args& a, const VirtualBlock& vb, char* smem) {
+    uint32_t* hist = reinterpret_cast<uint32_t*>(smem);
+    float* qx = reinterpret_cast<float*>(hist + kWarps * kMaxBins * 32);
+    float* qy = qx + kTile;
+    float* qz = qy + kTile;
+    float* edges = qz + kTile;
+    const int t = threadIdx.x, lane = t & 31, warp = t >> 5;
+    const uint32_t n = a.npts, S = a.nsets, ne = a.nedges;
+    const uint32_t s = vb.y;
+    const float* P;
+    const float* Q;
+    unsigned long long* out;
+    bool upper;
+    if (s == 0) {
+      P = Q = a.data;
+      out = a.dd;
+      upper = true;
+    } else if (s <= S) {
+      P = Q = a.rand + (size_t)(s - 1) * 3 * n;
+      out = a.rr;
+      upper = true;
+    } else {
+      P = a.data;
+      Q = a.rand + (size_t)(s - S - 1) * 3 * n;
+      out = a.dr;
+      upper = false;
+    }
+    for (int b = t; b < kWarps * kMaxBins * 32; b += kThreads) hist[b] = 0u;
+    if (t < 32) edges[t] = t < (int)ne ? __ldg(a.binb + t) : -3.0f;  // pad: never > d
+    const uint32_t i = vb.x * kTile + t;
+    const bool have = i < n;
+    const float ix = have ? __ldg(P + i) : 0.f, iy = have ? __ldg(P + n + i) : 0.f,
+                iz = have ? __ldg(P + 2 * n + i) : 0.f;
+    uint32_t* myh = hist + warp * kMaxBins * 32 + lane;
+    const uint32_t j_first_tile = upper ? vb.x * kTile : 0;
+    for (uint32_t jt = j_first_tile; jt < n; jt += kTile) {
+      __syncthreads();
+      const uint32_t jj = jt + t;
+      if (jj < n) {
+        qx[t] = __ldg(Q + jj);
+        qy[t] = __ldg(Q + n + jj);
+        qz[t] = __ldg(Q + 2 * n + jj);
+      }
+      __syncthreads();
+      if (!have) continue;
+      const uint32_t cnt = min((uint32_t)kTile, n - jt);
+      // pairs i < j on the diagonal tile start after i
+      const uint32_t q0 = (upper && jt == vb.x * kTile) ? (uint32_t)t + 1 : 0u;
+      for (uint32_t q = q0; q < cnt; ++q) {
+        const float d = __fadd_rn(__fadd_rn(__fmul_rn(ix, qx[q]), __fmul_rn(iy, qy[q])),
+                                  __fmul_rn(iz, qz[q]));
+        // bin = #{k : d < edges[k]}; edges descending -> binary search
+        int m = 0;
+#pragma unroll
+        for (int step = 16; step >= 1; step >>= 1)
+          if (edges[m + step - 1] > d) m += step;
+        myh[m * 32] += 1u;
+      }
+    }
+    __syncthreads();
+    if (t < (int)ne + 1) {
+      unsigned long long tot = 0;
+      for (int w = 0; w < kWarps; ++w)
+        for (int l = 0; l < 32; ++l) tot += hist[(w * kMaxBins + t) * 32 + l];
+      if (tot) atomicAdd(out + t, tot);
+    }
+  }
+};
+
+}  // namespace accel

@@ -200,7 +200,92 @@ class HistoJob(Job):
         return {"bytes": b * self.iters, "bytes_per_launch": b, "bound": "hbm", "launches": self.iters}
 
 
-JOBS = {"mop": MopJob, "stencil": StencilJob, "histo": HistoJob}
+class BfsJob(Job):
+    """One request = `levels` launches of the level-expansion kernel (upper
+    bound on the BFS depth; launches past the last level find an empty
+    frontier on the device and return immediately)."""
+
+    def __init__(self, d: dict, device="cuda", levels: int | None = None):
+        super().__init__(name="bfs", device=torch.device(device))
+        self.nv, self.ne, self.src = d["nv"], d["ne"], d["src"]
+        self.levels = levels or d.get("levels", 24)
+        self.inputs = {"row_ptr": _dev(d["row_ptr"], self.device), "col": _dev(d["col"], self.device)}
+        self.level = torch.empty(self.nv, dtype=torch.int32, device=self.device)
+        self.frontier = torch.empty(2 * self.nv, dtype=torch.int32, device=self.device)
+        self.count = torch.zeros(self.levels + 1, dtype=torch.int32, device=self.device)
+        self.out = {"level": self.level}
+        self.args = abi.accel_bfs_args(self.inputs["row_ptr"].data_ptr(), self.inputs["col"].data_ptr(),
+                                       self.nv, self.src, self.level.data_ptr(), self.frontier.data_ptr(),
+                                       self.count.data_ptr())
+        self.clears = [(self.level, 0xFF), (self.count, 0)]
+        self.steps = [Step("bfs", (_cdiv(self.nv, 256), 1, 1), self.args, self.levels)]
+
+    def result(self):
+        return {"level": _np(self.level, np.int32)}
+
+    def frontier_sizes(self):
+        return _np(self.count, np.uint32)
+
+    def work(self):
+        b = 16 * self.nv + 8 * self.ne
+        return {"bytes": b, "bytes_per_launch": b / self.levels, "bound": "hbm", "launches": self.levels}
+
+
+class CutcpJob(Job):
+    def __init__(self, d: dict, device="cuda"):
+        super().__init__(name="cutcp", device=torch.device(device))
+        self.d = {k: d[k] for k in ("nx", "ny", "nz", "h", "cutoff", "excl", "natoms", "box")}
+        self.nx, self.ny, self.nz = d["nx"], d["ny"], d["nz"]
+        self.inputs = {"atoms": _dev(d["atoms"].ravel(), self.device),
+                       "cell_start": _dev(d["cell_start"], self.device)}
+        self.v = torch.empty(self.nz * self.ny * self.nx, dtype=torch.float32, device=self.device)
+        self.out = {"v": self.v}
+        self.args = abi.accel_cutcp_args(self.inputs["atoms"].data_ptr(), self.inputs["cell_start"].data_ptr(),
+                                         d["ncell_1d"], d["cell"], self.nx, self.ny, self.nz, d["h"],
+                                         d["cutoff"], d["excl"], self.v.data_ptr())
+        self.steps = [Step("cutcp", (_cdiv(self.nx, 8), _cdiv(self.ny, 8), _cdiv(self.nz, 8)), self.args, 1)]
+
+    def result(self):
+        return {"v": _np(self.v, np.float32).reshape(self.nz, self.ny, self.nx)}
+
+    def work(self):
+        # in-cutoff (lattice point, atom) pairs, estimated from the mean atom
+        # density (DESIGN.md: cutcp algorithmic work); ~15 flop each
+        dens = self.d["natoms"] / self.d["box"] ** 3
+        pairs = self.nx * self.ny * self.nz * dens * 4.0 / 3.0 * np.pi * self.d["cutoff"] ** 3
+        return {"pairs": pairs, "flops": 15.0 * pairs, "bound": "alu", "launches": 1}
+
+
+class TpacfJob(Job):
+    def __init__(self, d: dict, device="cuda"):
+        super().__init__(name="tpacf", device=torch.device(device))
+        self.n, self.S = d["npts"], d["nsets"]
+        self.nedges = len(d["binb"])
+        assert self.nedges + 1 <= 32
+        self.inputs = {"data": _dev(d["data"], self.device), "rand": _dev(d["rand"], self.device),
+                       "binb": _dev(d["binb"], self.device)}
+        nb = self.nedges + 1
+        self.hists = torch.zeros(3 * nb, dtype=torch.int64, device=self.device)
+        self.out = {"hists": self.hists}
+        p = self.hists.data_ptr()
+        self.args = abi.accel_tpacf_args(self.inputs["data"].data_ptr(), self.inputs["rand"].data_ptr(),
+                                         self.inputs["binb"].data_ptr(), self.n, self.S, self.nedges,
+                                         p, p + 8 * nb, p + 16 * nb)
+        self.clears = [(self.hists, 0)]
+        self.steps = [Step("tpacf", (_cdiv(self.n, 256), 2 * self.S + 1, 1), self.args, 1)]
+
+    def result(self):
+        h = _np(self.hists, np.uint64).reshape(3, -1)
+        return {"dd": h[0], "rr": h[1], "dr": h[2]}
+
+    def work(self):
+        n, S = self.n, self.S
+        pairs = (1 + S) * n * (n - 1) // 2 + S * n * n
+        return {"pairs": pairs, "flops": 5.0 * pairs, "bound": "alu", "launches": 1}
+
+
+JOBS = {"mop": MopJob, "stencil": StencilJob, "histo": HistoJob, "bfs": BfsJob, "cutcp": CutcpJob,
+        "tpacf": TpacfJob}
 
 
 def make_job(name: str, d: dict, device="cuda") -> Job:

@@ -68,6 +68,9 @@ class Accel:
     def stats(self, rid: int) -> abi.accel_req_stats:
         return abi.accel_stats(self.ctx, rid)
 
+    def launch_stats(self, rid: int, n: int) -> list[abi.accel_launch_stat]:
+        return abi.accel_launch_stats(self.ctx, rid, n)
+
     def launch_times(self, rid: int, n: int) -> list[float]:
         return abi.accel_launch_times(self.ctx, rid, n)
 

@@ -1,0 +1,3 @@
+set -x
+timeout 1200 python -m pytest tests -m gpu -x -q 2>&1 | tail -15
+timeout 900 python bench.py --steps 5 --warmup 3 --out gpurun_out/bench_c2_resolve.json 2>&1 | tail -3

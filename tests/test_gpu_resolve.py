@@ -1,0 +1,97 @@
+"""GPU: the RESOLVE policy (quota re-solve on arrival and departure,
+BASELINE.json north star) -- shrink through the live-quota word, growth through
+sticky top-up grids -- keeps every result exact and every VG covered once."""
+import time
+
+import numpy as np
+import pytest
+
+import synth
+from tests.gpu_util import assert_close_fp32
+
+pytestmark = pytest.mark.gpu
+
+
+@pytest.fixture(scope="module")
+def racc():
+    import torch
+    if not torch.cuda.is_available():
+        pytest.skip("no GPU")
+    from paper_conf_cgo_margiolaso16_b200 import abi
+    from paper_conf_cgo_margiolaso16_b200.runtime import Accel
+    a = Accel(device=0, mode=abi.MODE_SHARED, policy=abi.POLICY_RESOLVE, verify=True)
+    yield a
+    a.close()
+
+
+def test_departure_grows_survivor(racc, oracle_lib):
+    """A short request (mop) leaves early; the long stencil grows into its share."""
+    from paper_conf_cgo_margiolaso16_b200.jobs import MopJob, StencilJob
+    ds = synth.preset("stencil", "default", seed=2, sweeps=60)
+    dm = synth.preset("mop", "small", seed=3)
+    js, jm = StencilJob(ds), MopJob(dm)
+    racc.run([js, jm])  # warm: module loading, first-touch
+    st = racc.run([js, jm])
+    assert all(s.coverage_ok == 1 for s in st)
+    assert np.array_equal(jm.result()["out"], oracle_lib.mop(dm))
+    s_st = st[0]
+    assert s_st.resolves >= 1 and s_st.quota_max > s_st.quota_initial, (
+        s_st.quota_initial, s_st.quota_max, s_st.resolves)
+    # sampled planes (light cone) vs the oracle
+    got = js.result()["a"]
+    zlo, zhi = 0, 64
+    ref = oracle_lib.stencil(dict(ds, sweeps=60))
+    assert_close_fp32(got[zlo:zhi:16], ref[zlo:zhi:16], what="stencil after growth")
+
+
+def test_arrival_shrinks_running(racc, oracle_lib):
+    """A running request shrinks when a second one arrives (staggered submit)."""
+    from paper_conf_cgo_margiolaso16_b200.jobs import CutcpJob, HistoJob
+    dc = synth.preset("cutcp", "default", seed=1)
+    dh = synth.preset("histo", "default", seed=2, iters=10)
+    jc, jh = CutcpJob(dc), HistoJob(dh)
+    ida = racc.submit([jc], tenants=[0])
+    time.sleep(0.0003)
+    idb = racc.submit([jh], tenants=[1])
+    racc.sync()
+    sa, sb = racc.stats(ida[0]), racc.stats(idb[0])
+    racc.release()
+    assert sa.coverage_ok == 1 and sb.coverage_ok == 1
+    assert sa.quota_min < sa.quota_initial or sa.last_end_ns < sb.first_start_ns
+    counts, _ = oracle_lib.histo(dh)
+    assert np.array_equal(jh.result()["counts"], counts)
+    r = np.random.Generator(np.random.PCG64(3))
+    ijk = np.stack([r.integers(0, dc["nx"], 500), r.integers(0, dc["ny"], 500), r.integers(0, dc["nz"], 500)], 1)
+    v = jc.result()["v"][ijk[:, 2], ijk[:, 1], ijk[:, 0]]
+    assert_close_fp32(v, oracle_lib.cutcp_points(dc, ijk), what="cutcp under shrink")
+
+
+@pytest.mark.parametrize("seed", [0, 1])
+def test_staggered_multi_launch_mix(racc, oracle_lib, seed):
+    """Config-4-like: several tenants arrive staggered, each re-solve shrinks
+    or grows the others, multi-launch requests (bfs levels, histo iterations,
+    stencil sweeps) stay correct."""
+    from paper_conf_cgo_margiolaso16_b200.jobs import BfsJob, HistoJob, StencilJob, TpacfJob
+    dsn = synth.preset("stencil", "default", seed=seed, sweeps=30)
+    dbf = synth.preset("bfs", "default", seed=seed)
+    dhi = synth.preset("histo", "default", seed=seed, iters=8)
+    dtp = synth.preset("tpacf", "small", seed=seed)
+    jobs = [StencilJob(dsn), BfsJob(dbf), HistoJob(dhi), TpacfJob(dtp)]
+    ids = []
+    for t, j in enumerate(jobs):
+        ids += racc.submit([j], tenants=[t])
+        time.sleep(0.0002)
+    racc.sync()
+    st = [racc.stats(i) for i in ids]
+    racc.release()
+    assert all(s.coverage_ok == 1 for s in st)
+    assert sum(s.resolves for s in st) >= 1
+    assert np.array_equal(jobs[1].result()["level"], oracle_lib.bfs(dbf)[0])
+    assert np.array_equal(jobs[2].result()["counts"], oracle_lib.histo(dhi)[0])
+    dd, rr, dr = oracle_lib.tpacf(dtp)
+    r = jobs[3].result()
+    assert np.array_equal(r["dd"], dd) and np.array_equal(r["rr"], rr) and np.array_equal(r["dr"], dr)
+    zlo, zhi = 10, 54  # planes 40..43 depend on [10, 74) ∩ [0, 64) after 30 sweeps
+    slab = dict(dsn, a0=np.ascontiguousarray(dsn["a0"][zlo:]), nz=64 - zlo)
+    ref = oracle_lib.stencil(slab)
+    assert_close_fp32(jobs[0].result()["a"][40:44], ref[40 - zlo:44 - zlo], what="stencil")

@@ -179,3 +179,100 @@ def test_quota_matches_occupancy_for_single_tenant(acc):
     g = int(np.prod(job.steps[0].grid))
     assert st.quota_initial == min(g, sms * info.occ_persistent)
     assert info.occ_persistent == info.occ_native
+
+
+# ---------------------------------------------------------------- bfs
+@pytest.mark.parametrize("size,over", [("tiny", {}), ("small", dict(seed=3)), ("small", dict(src=17, seed=5)),
+                                       ("tiny", dict(deg_lo=0, deg_hi=2, seed=9))])
+def test_bfs(acc_tiny_caps, oracle_lib, size, over):
+    from paper_conf_cgo_margiolaso16_b200.jobs import BfsJob
+    d = synth.preset("bfs", size, **over)
+    ref, depth = oracle_lib.bfs(d)
+    levels = depth + 3  # more launches than levels: empty frontiers must be no-ops
+    nat, sh, _ = run_modes(acc_tiny_caps, lambda: BfsJob(d, levels=levels))
+    assert np.array_equal(nat["level"], ref)
+    assert np.array_equal(sh["level"], ref)
+
+
+def test_bfs_default(acc, oracle_lib):
+    from paper_conf_cgo_margiolaso16_b200.jobs import BfsJob
+    d = synth.preset("bfs", "default")
+    ref, depth = oracle_lib.bfs(d)
+    assert depth + 1 < 24  # the bench's launch count covers every level
+    nat, sh, _ = run_modes(acc, lambda: BfsJob(d))
+    assert np.array_equal(nat["level"], ref) and np.array_equal(sh["level"], ref)
+
+
+# ---------------------------------------------------------------- cutcp
+@pytest.mark.parametrize("size,over", [("tiny", {}), ("tiny", dict(seed=5, box=24.0)), ("small", {})])
+def test_cutcp(acc_tiny_caps, oracle_lib, size, over):
+    from paper_conf_cgo_margiolaso16_b200.jobs import CutcpJob
+    d = synth.preset("cutcp", size, **over)
+    nat, sh, _ = run_modes(acc_tiny_caps, lambda: CutcpJob(d))
+    same(nat, sh)
+    ref = oracle_lib.cutcp(d)
+    assert np.array_equal(sh["v"] == 0, ref == 0)  # exclusion decided identically
+    assert_close_fp32(sh["v"], ref, what="cutcp")
+
+
+def test_cutcp_default_sampled(acc, oracle_lib):
+    from paper_conf_cgo_margiolaso16_b200.jobs import CutcpJob
+    d = synth.preset("cutcp", "default")
+    job = CutcpJob(d)
+    acc.run([job])
+    v = job.result()["v"]
+    r = np.random.Generator(np.random.PCG64(1))
+    ijk = np.stack([r.integers(0, d["nx"], 3000), r.integers(0, d["ny"], 3000), r.integers(0, d["nz"], 3000)], 1)
+    ref = oracle_lib.cutcp_points(d, ijk)
+    got = v[ijk[:, 2], ijk[:, 1], ijk[:, 0]]
+    assert np.array_equal(got == 0, ref == 0)
+    assert_close_fp32(got, ref, what="cutcp default")
+
+
+# ---------------------------------------------------------------- tpacf
+@pytest.mark.parametrize("size,over", [("tiny", {}), ("small", {}), ("tiny", dict(npts=257, nsets=2))])
+def test_tpacf(acc_tiny_caps, oracle_lib, size, over):
+    from paper_conf_cgo_margiolaso16_b200.jobs import TpacfJob
+    d = synth.preset("tpacf", size, **over)
+    nat, sh, _ = run_modes(acc_tiny_caps, lambda: TpacfJob(d))
+    dd, rr, dr = oracle_lib.tpacf(d)
+    for r in (nat, sh):
+        assert np.array_equal(r["dd"], dd) and np.array_equal(r["rr"], rr) and np.array_equal(r["dr"], dr)
+
+
+def test_tpacf_default(acc, oracle_lib):
+    from paper_conf_cgo_margiolaso16_b200.jobs import TpacfJob
+    d = synth.preset("tpacf", "default")
+    job = TpacfJob(d)
+    acc.run([job])
+    dd, rr, dr = oracle_lib.tpacf(d)
+    r = job.result()
+    assert np.array_equal(r["dd"], dd) and np.array_equal(r["rr"], rr) and np.array_equal(r["dr"], dr)
+
+
+# ---------------------------------------------------------------- config 2
+def test_config2_fig2_mix(acc, oracle_lib):
+    """Fig. 2 mix (bfs + cutcp + stencil + tpacf) at bench sizes, both modes:
+    outputs under concurrency equal the isolated oracle results."""
+    from paper_conf_cgo_margiolaso16_b200 import abi
+    from paper_conf_cgo_margiolaso16_b200.jobs import make_job
+    names = ["bfs", "cutcp", "stencil", "tpacf"]
+    ds = {"bfs": synth.preset("bfs", "default", seed=3),
+          "cutcp": synth.preset("cutcp", "small", seed=4),
+          "stencil": synth.preset("stencil", "small", seed=5, sweeps=10),
+          "tpacf": synth.preset("tpacf", "small", seed=6)}
+    refs = {"bfs": oracle_lib.bfs(ds["bfs"])[0], "cutcp": oracle_lib.cutcp(ds["cutcp"]),
+            "stencil": oracle_lib.stencil(ds["stencil"]), "tpacf": oracle_lib.tpacf(ds["tpacf"])}
+    for mode in (abi.MODE_SHARED, abi.MODE_NATIVE):
+        acc.set_mode(mode)
+        jobs = [make_job(n, ds[n]) for n in names]
+        st = acc.run(jobs)
+        assert all(s.coverage_ok == 1 for s in st)
+        assert np.array_equal(jobs[0].result()["level"], refs["bfs"])
+        assert_close_fp32(jobs[1].result()["v"], refs["cutcp"])
+        assert_close_fp32(jobs[2].result()["a"], refs["stencil"])
+        r = jobs[3].result()
+        assert np.array_equal(r["dd"], refs["tpacf"][0]) and np.array_equal(r["dr"], refs["tpacf"][2])
+        if mode == abi.MODE_SHARED:
+            assert len({s.quota_initial for s in st}) >= 1
+    acc.set_mode(abi.MODE_SHARED)
