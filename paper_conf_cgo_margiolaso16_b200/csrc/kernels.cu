@@ -11,6 +11,9 @@
 #include "tenants/cutcp.cuh"
 #include "tenants/histo.cuh"
 #include "tenants/mop.cuh"
+#include "tenants/mriq.cuh"
+#include "tenants/sgemm.cuh"
+#include "tenants/spmv.cuh"
 #include "tenants/stencil.cuh"
 #include "tenants/tpacf.cuh"
 
@@ -95,6 +98,10 @@ const Builtin kBuiltins[] = {
     {"bfs", &make_desc<Bfs>},
     {"cutcp", &make_desc<Cutcp>},
     {"tpacf", &make_desc<Tpacf>},
+    {"spmv", &make_desc<Spmv>},
+    {"sgemm", &make_desc<Sgemm>},
+    {"mriq_phimag", &make_desc<MriqPhiMag>},
+    {"mriq_q", &make_desc<MriqQ>},
 };
 constexpr int kNumBuiltins = sizeof(kBuiltins) / sizeof(kBuiltins[0]);
 }  // namespace

@@ -1,0 +1,90 @@
+// mri-q -- non-Cartesian MRI reconstruction Q matrix (Parboil "mri-q":
+// ComputePhiMag + ComputeQ).
+//
+// ComputePhiMag: phiMag_k = phiR^2 + phiI^2 (fp32, round-to-nearest, no FMA:
+// bit-exact vs the oracle).  ComputeQ: Qr + i Qi = sum_k phiMag_k
+// exp(2 pi i (kx x + ky y + kz z)).  One VG = 256 voxels, one per thread; the
+// k-samples are staged through shared memory in tiles of 256.  The phase is
+// reduced exactly in "turns": every product k_d * x_d is split into its fp32
+// value p and its FMA residual e (p + e exact), p - rint(p) is exact, so
+// t = frac(sum) is accurate to ~1e-7 turns although |k.x| reaches ~90 turns
+// (plain fp32 would give ~5e-4 relative error in Q, DESIGN.md R-fp-2); then
+// one MUFU sin/cos pair.  SFU/ALU-bound.
+#pragma once
+#include "../device/dispatch.cuh"
+#include "accel_tenants.h"
+
+namespace accel {
+
+struct MriqPhiMag {
+  using Args = accel_mriq_phimag_args;
+  static constexpr int kThreads = 256;
+  static constexpr uint32_t kChunk = 4;
+  static constexpr int kMinBlocks = 8;
+  static constexpr uint32_t kDynSmem = 0;
+  static __device__ __forceinline__ void body(const Args& a, const VirtualBlock& vb, char*) {
+    const uint32_t k = vb.linear * kThreads + threadIdx.x;
+    if (k >= a.numk) return;
+    const float r = a.phir[k], i = a.phii[k];
+    a.phimag[k] = __fadd_rn(__fmul_rn(r, r), __fmul_rn(i, i));
+  }
+};
+
+struct MriqQ {
+  using Args = accel_mriq_q_args;
+  static constexpr int kThreads = 256;
+  static constexpr int kTile = 256;
+  static constexpr uint32_t kChunk = 1;
+  static constexpr int kMinBlocks = 6;
+  static constexpr uint32_t kDynSmem = 4 * kTile * sizeof(float);
+
+  static __device__ __forceinline__ float frac_prod(float k, float x, float& err) {
+    const float p = __fmul_rn(k, x);  // no contraction: p + residual == k*x exactly
+    err += __fmaf_rn(k, x, -p);       // exact residual of the product
+    return __fsub_rn(p, rintf(p));    // exact
+  }
+
+  static __device__ __forceinline__ void body(const Args& a, const VirtualBlock& vb, char* smem) {
+    float* skx = reinterpret_cast<float*>(smem);
+    float* sky = skx + kTile;
+    float* skz = sky + kTile;
+    float* spm = skz + kTile;
+    const int t = threadIdx.x;
+    const uint32_t v = vb.linear * kThreads + t;
+    const bool have = v < a.numx;
+    const float x = have ? __ldg(a.x + v) : 0.f;
+    const float y = have ? __ldg(a.y + v) : 0.f;
+    const float z = have ? __ldg(a.z + v) : 0.f;
+    float qr = 0.f, qi = 0.f;
+    const float two_pi = 6.2831853071795864769f;
+    for (uint32_t k0 = 0; k0 < a.numk; k0 += kTile) {
+      __syncthreads();
+      const uint32_t k = k0 + t;
+      if (k < a.numk) {
+        skx[t] = __ldg(a.kx + k);
+        sky[t] = __ldg(a.ky + k);
+        skz[t] = __ldg(a.kz + k);
+        spm[t] = __ldcg(a.phimag + k);   // written by the previous launch
+      }
+      __syncthreads();
+      const int n = min(kTile, (int)(a.numk - k0));
+#pragma unroll 4
+      for (int j = 0; j < n; ++j) {
+        float err = 0.f;
+        const float f = frac_prod(skx[j], x, err) + frac_prod(sky[j], y, err) + frac_prod(skz[j], z, err);
+        float tt = f + err;
+        tt -= rintf(tt);                 // turns in [-0.5, 0.5]
+        float s, c;
+        __sincosf(two_pi * tt, &s, &c);
+        qr = fmaf(spm[j], c, qr);
+        qi = fmaf(spm[j], s, qi);
+      }
+    }
+    if (have) {
+      a.qr[v] = qr;
+      a.qi[v] = qi;
+    }
+  }
+};
+
+}  // namespace accel

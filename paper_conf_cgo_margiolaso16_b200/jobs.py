@@ -284,8 +284,79 @@ class TpacfJob(Job):
         return {"pairs": pairs, "flops": 5.0 * pairs, "bound": "alu", "launches": 1}
 
 
+class SpmvJob(Job):
+    def __init__(self, d: dict, device="cuda"):
+        super().__init__(name="spmv", device=torch.device(device))
+        self.n, self.nnz, self.iters = d["n"], d["nnz"], d["iters"]
+        self.inputs = {k: _dev(d[k], self.device) for k in ("row_ptr", "col", "val", "x")}
+        self.y = torch.empty(self.n, dtype=torch.float32, device=self.device)
+        self.out = {"y": self.y}
+        i = self.inputs
+        self.args = abi.accel_spmv_args(i["row_ptr"].data_ptr(), i["col"].data_ptr(), i["val"].data_ptr(),
+                                        i["x"].data_ptr(), self.y.data_ptr(), self.n)
+        self.steps = [Step("spmv", (_cdiv(self.n, 64), 1, 1), self.args, self.iters)]
+
+    def result(self):
+        return {"y": _np(self.y, np.float32)}
+
+    def work(self):
+        b = 8 * self.nnz + 12 * self.n
+        return {"bytes": b * self.iters, "bytes_per_launch": b, "bound": "hbm", "launches": self.iters}
+
+
+class SgemmJob(Job):
+    def __init__(self, d: dict, device="cuda"):
+        super().__init__(name="sgemm", device=torch.device(device))
+        self.m, self.n, self.k = d["m"], d["n"], d["k"]
+        if self.k % 4:
+            raise ValueError("sgemm needs k % 4 == 0 (16-B rows)")
+        self.inputs = {"a": _dev(d["a"].ravel(), self.device), "b": _dev(d["b"].ravel(), self.device)}
+        self.c = torch.empty(self.m * self.n, dtype=torch.float32, device=self.device)
+        self.out = {"c": self.c}
+        self.args = abi.accel_sgemm_args(self.inputs["a"].data_ptr(), self.inputs["b"].data_ptr(),
+                                         self.c.data_ptr(), self.m, self.n, self.k)
+        self.steps = [Step("sgemm", (_cdiv(self.n, 128), _cdiv(self.m, 128), 1), self.args, 1)]
+
+    def result(self):
+        return {"c": _np(self.c, np.float32).reshape(self.m, self.n)}
+
+    def work(self):
+        f = 2.0 * self.m * self.n * self.k
+        return {"flops": f, "flops_per_launch": f, "bound": "alu", "launches": 1}
+
+
+class MriqJob(Job):
+    """Two steps, like Parboil's mri-q: ComputePhiMag (tiny) then ComputeQ."""
+
+    def __init__(self, d: dict, device="cuda"):
+        super().__init__(name="mriq", device=torch.device(device))
+        self.numx, self.numk = d["numx"], d["numk"]
+        self.inputs = {k: _dev(d[k], self.device) for k in ("kx", "ky", "kz", "phir", "phii", "x", "y", "z")}
+        i = self.inputs
+        self.phimag = torch.empty(self.numk, dtype=torch.float32, device=self.device)
+        self.qr = torch.empty(self.numx, dtype=torch.float32, device=self.device)
+        self.qi = torch.empty(self.numx, dtype=torch.float32, device=self.device)
+        self.out = {"phimag": self.phimag, "qr": self.qr, "qi": self.qi}
+        self.args_pm = abi.accel_mriq_phimag_args(i["phir"].data_ptr(), i["phii"].data_ptr(),
+                                                  self.phimag.data_ptr(), self.numk)
+        self.args_q = abi.accel_mriq_q_args(i["kx"].data_ptr(), i["ky"].data_ptr(), i["kz"].data_ptr(),
+                                            self.phimag.data_ptr(), self.numk, self.numx, i["x"].data_ptr(),
+                                            i["y"].data_ptr(), i["z"].data_ptr(), self.qr.data_ptr(),
+                                            self.qi.data_ptr())
+        self.steps = [Step("mriq_phimag", (_cdiv(self.numk, 256), 1, 1), self.args_pm, 1),
+                      Step("mriq_q", (_cdiv(self.numx, 256), 1, 1), self.args_q, 1)]
+
+    def result(self):
+        return {k: _np(t, np.float32) for k, t in self.out.items()}
+
+    def work(self):
+        pairs = self.numx * self.numk
+        return {"pairs": pairs, "flops": 11.0 * pairs, "sfu": 2 * pairs, "bound": "alu", "launches": 2,
+                "skip_launches": 1, "flops_per_launch": 11.0 * pairs}
+
+
 JOBS = {"mop": MopJob, "stencil": StencilJob, "histo": HistoJob, "bfs": BfsJob, "cutcp": CutcpJob,
-        "tpacf": TpacfJob}
+        "tpacf": TpacfJob, "spmv": SpmvJob, "sgemm": SgemmJob, "mriq": MriqJob}
 
 
 def make_job(name: str, d: dict, device="cuda") -> Job:

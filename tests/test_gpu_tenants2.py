@@ -1,0 +1,89 @@
+"""GPU parity for spmv, sgemm and mri-q (both modes, coverage, oracle)."""
+import numpy as np
+import pytest
+
+import synth
+from tests.gpu_util import assert_close_fp32
+from tests.test_gpu_tenants import acc, acc_tiny_caps, run_modes, same  # noqa: F401  (fixtures)
+
+pytestmark = pytest.mark.gpu
+
+
+@pytest.mark.parametrize("size,over", [("tiny", {}), ("small", dict(iters=3)), ("tiny", dict(grid=7, reach=3))])
+def test_spmv(acc_tiny_caps, oracle_lib, size, over):
+    from paper_conf_cgo_margiolaso16_b200.jobs import SpmvJob
+    d = synth.preset("spmv", size, **over)
+    nat, sh, _ = run_modes(acc_tiny_caps, lambda: SpmvJob(d))
+    same(nat, sh)
+    assert_close_fp32(sh["y"], oracle_lib.spmv(d), what="spmv")
+
+
+def test_spmv_default(acc, oracle_lib):
+    from paper_conf_cgo_margiolaso16_b200.jobs import SpmvJob
+    d = synth.preset("spmv", "default", iters=2)
+    nat, sh, _ = run_modes(acc, lambda: SpmvJob(d))
+    same(nat, sh)
+    assert_close_fp32(sh["y"], oracle_lib.spmv(d), what="spmv default")
+
+
+@pytest.mark.parametrize("size,over", [("tiny", {}), ("small", {}), ("tiny", dict(m=129, n=257, k=36))])
+def test_sgemm(acc_tiny_caps, oracle_lib, size, over):
+    from paper_conf_cgo_margiolaso16_b200.jobs import SgemmJob
+    d = synth.preset("sgemm", size, **over)
+    nat, sh, _ = run_modes(acc_tiny_caps, lambda: SgemmJob(d))
+    same(nat, sh)
+    assert_close_fp32(sh["c"], oracle_lib.sgemm(d), what="sgemm")
+
+
+def test_sgemm_default_sampled(acc, oracle_lib):
+    from paper_conf_cgo_margiolaso16_b200.jobs import SgemmJob
+    d = synth.preset("sgemm", "default")
+    job = SgemmJob(d)
+    acc.run([job])
+    c = job.result()["c"]
+    r = np.random.Generator(np.random.PCG64(2))
+    ij = np.stack([r.integers(0, d["m"], 4000), r.integers(0, d["n"], 4000)], 1)
+    ij = np.concatenate([ij, [[0, 0], [d["m"] - 1, d["n"] - 1], [127, 128], [128, 127]]])
+    assert_close_fp32(c[ij[:, 0], ij[:, 1]], oracle_lib.sgemm_entries(d, ij), what="sgemm default")
+
+
+def test_sgemm_identity():
+    """B = I reproduces A (within fp32 rounding of a single product)."""
+    import torch
+    if not torch.cuda.is_available():
+        pytest.skip("no GPU")
+    from paper_conf_cgo_margiolaso16_b200.jobs import SgemmJob
+    from paper_conf_cgo_margiolaso16_b200.runtime import Accel
+    k = 256
+    a = synth.preset("sgemm", "tiny", k=k)["a"]
+    d = {"a": a, "b": np.eye(k, dtype=np.float32), "m": a.shape[0], "n": k, "k": k}
+    with Accel(0) as acc:
+        job = SgemmJob(d)
+        acc.run([job])
+        assert np.array_equal(job.result()["c"], a)
+
+
+@pytest.mark.parametrize("size,over", [("tiny", {}), ("small", dict(numk=1000)), ("tiny", dict(nvox_1d=7, numk=257))])
+def test_mriq(acc_tiny_caps, oracle_lib, size, over):
+    from paper_conf_cgo_margiolaso16_b200.jobs import MriqJob
+    d = synth.preset("mriq", size, **over)
+    nat, sh, _ = run_modes(acc_tiny_caps, lambda: MriqJob(d))
+    same(nat, sh)
+    pm, qr, qi = oracle_lib.mriq(d)
+    assert np.array_equal(sh["phimag"], pm)
+    assert_close_fp32(np.concatenate([sh["qr"], sh["qi"]]), np.concatenate([qr, qi]), what="mri-q")
+
+
+def test_mriq_default_sampled(acc, oracle_lib):
+    from paper_conf_cgo_margiolaso16_b200.jobs import MriqJob
+    d = synth.preset("mriq", "default")
+    job = MriqJob(d)
+    acc.run([job])
+    res = job.result()
+    pm = oracle_lib.mriq_phimag(d)
+    assert np.array_equal(res["phimag"], pm)
+    r = np.random.Generator(np.random.PCG64(5))
+    idx = np.concatenate([r.integers(0, d["numx"], 1500), [0, d["numx"] - 1]])
+    qr, qi = oracle_lib.mriq_points(d, idx, pm)
+    assert_close_fp32(np.concatenate([res["qr"][idx], res["qi"][idx]]), np.concatenate([qr, qi]),
+                      what="mri-q default")
