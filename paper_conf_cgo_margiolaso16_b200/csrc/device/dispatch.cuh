@@ -49,30 +49,49 @@ struct Ctl {
 };
 
 // Virtual NDRange of ONE launch ("Virtual Kernel Execution
-// Range which is copied to the accelerator memory").  256 B: read-mostly
-// fields and stamps, then the hot dequeue counter on its own 128-B line.
+// Range which is copied to the accelerator memory").  384 B = three 128-B
+// lines so that the three access patterns never share a line (an L2 line that
+// takes atomics serialises every other access to it; measured):
+//   line 0  read-only during the launch (written by the init kernel) -> L1 hits
+//   line 1  the software queue head (one atomicAdd per dequeue)
+//   line 2  statistics and RESOLVE admission (reductions, rare atomics)
 struct alignas(128) Desc {
+  // ---- line 0
   uint32_t total;        // VGs in the original grid (static upper bound)
   uint32_t gx, gy, gz;   // original grid shape (decode, R-disp-2)
   uint32_t chunk;        // VGs per dequeue (§6.4)
   uint32_t launch_idx;   // index of this launch inside its step
   uint32_t flags;        // kFlag*
-  uint32_t total_seen;   // total as read by the CTAs (dynamic for bfs)
+  uint32_t req_idx;      // launch index inside the request
   Ctl* ctl;              // RESOLVE control block, nullptr otherwise
   uint32_t* coverage;    // verify: coverage[vg] += 1
-  unsigned long long t_first;  // min %globaltimer over CTA starts
-  unsigned long long t_last;   // max %globaltimer over CTA ends
-  uint32_t ctas_started; // CTAs admitted with work
-  uint32_t alive;        // CTAs currently admitted
-  uint32_t max_alive;    // high-water mark of `alive`
-  uint32_t topped;       // a top-up CTA joined this launch
-  uint32_t req_idx;      // launch index inside the request
   uint32_t has_prev;     // this - 1 is the request's previous launch
+  uint32_t pad0[19];
   // ---- line 1: the software queue head (RUN_TERMINATE when >= total)
   uint32_t next;
   uint32_t pad1[31];
+  // ---- line 2
+  unsigned long long t_first;  // min %globaltimer over CTA starts
+  unsigned long long t_last;   // max %globaltimer over CTA ends
+  uint32_t total_seen;   // total as read by the CTAs (dynamic for bfs)
+  uint32_t ctas_started; // CTAs admitted with work
+  uint32_t alive;        // CTAs currently admitted (RESOLVE)
+  uint32_t max_alive;    // high-water mark of `alive` (RESOLVE)
+  uint32_t topped;       // a top-up CTA joined this launch (RESOLVE)
+  uint32_t pad2[23];
 };
-static_assert(sizeof(Desc) == 256, "Desc layout");
+static_assert(sizeof(Desc) == 384, "Desc layout");
+
+// Fire-and-forget reductions (no return value, no round trip).
+__device__ __forceinline__ void red_min_u64(unsigned long long* p, unsigned long long v) {
+  asm volatile("red.relaxed.gpu.global.min.u64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
+}
+__device__ __forceinline__ void red_max_u64(unsigned long long* p, unsigned long long v) {
+  asm volatile("red.relaxed.gpu.global.max.u64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
+}
+__device__ __forceinline__ void red_add_u32(uint32_t* p, uint32_t v) {
+  asm volatile("red.relaxed.gpu.global.add.u32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
+}
 
 enum : uint32_t { kFlagStamps = 1u, kFlagAlive = 2u };
 
@@ -156,32 +175,39 @@ __device__ __forceinline__ void wait_complete(const Desc* p) {
   __threadfence();
 }
 
-// Master work-item, admission into launch d: count-based under RESOLVE,
-// plain alive tracking otherwise.  Returns false if the CTA must not work on d.
-__device__ __forceinline__ bool admit(Desc* d, uint32_t flags) {
-  const Ctl* ctl = d->ctl;
-  if (ctl != nullptr) {
-    const uint32_t a = atomicAdd(&d->alive, 1u) + 1u;
-    if (a > ld_volatile(&ctl->live)) {
-      atomicSub(&d->alive, 1u);
-      return false;
-    }
-    atomicMax(&d->max_alive, a);
-    __threadfence();  // admission visible before the first dequeue
-  } else if (flags & kFlagAlive) {
-    const uint32_t a = atomicAdd(&d->alive, 1u) + 1u;
-    atomicMax(&d->max_alive, a);
+// Launch configuration word, a kernel parameter (no descriptor load on the
+// critical path of a CTA's first dequeue): bits 0-15 chunk, then flags.
+//   kCfgDepth2: two dequeues in flight per CTA (the next VG id is requested
+//               two VGs ahead, hiding atomic latency behind long VG bodies).
+//   kCfgStride: static round-robin VG assignment (VG = cta + i * grid), no
+//               queue -- an ablation to measure the cost of the dynamic queue.
+enum : uint32_t {
+  kCfgChunkMask = 0xffffu,
+  kCfgResolve = 1u << 16,
+  kCfgStamps = 1u << 17,
+  kCfgDepth2 = 1u << 18,
+  kCfgStride = 1u << 19
+};
+
+// Master work-item, admission into launch d under RESOLVE (count-based):
+// returns false if the launch already holds `live` CTAs.
+__device__ __forceinline__ bool admit(Desc* d) {
+  const uint32_t a = atomicAdd(&d->alive, 1u) + 1u;
+  if (a > ld_volatile(&d->ctl->live)) {
+    atomicSub(&d->alive, 1u);
+    return false;
   }
+  atomicMax(&d->max_alive, a);
+  __threadfence();  // admission visible before the first dequeue
   return true;
 }
 
 // One dequeue (Fig. 8b line 26, rt_sched_wgroup): under RESOLVE a CTA
 // leaves first if the launch holds more CTAs than the live quota (shrink at a
 // VG boundary); then one atomicAdd of `chunk` on the queue head.
-__device__ __forceinline__ uint32_t dequeue(Desc* d, uint32_t chunk, bool& admitted) {
-  const Ctl* ctl = d->ctl;
-  if (ctl != nullptr) {
-    const uint32_t live = ld_volatile(&ctl->live);
+__device__ __forceinline__ uint32_t dequeue(Desc* d, uint32_t chunk, bool resolve, bool& admitted) {
+  if (resolve) {
+    const uint32_t live = ld_volatile(&d->ctl->live);
     if (ld_volatile(&d->alive) > live) {
       if (atomicSub(&d->alive, 1u) > live) {
         admitted = false;
@@ -193,38 +219,46 @@ __device__ __forceinline__ uint32_t dequeue(Desc* d, uint32_t chunk, bool& admit
   return atomicAdd(&d->next, chunk);
 }
 
-__device__ __forceinline__ void retire(Desc* d, uint32_t flags, bool admitted) {
-  if (admitted && (d->ctl != nullptr || (flags & kFlagAlive))) {
+__device__ __forceinline__ void retire(Desc* d, uint32_t cfg, bool admitted) {
+  if ((cfg & kCfgResolve) && admitted) {
     __threadfence();  // this CTA's VG results before the alive decrement
     atomicSub(&d->alive, 1u);
   }
-  if (flags & kFlagStamps) atomicMax(&d->t_last, globaltimer());
+  if (cfg & kCfgStamps) red_max_u64(&d->t_last, globaltimer());
 }
 
 // Serve one launch: admission, dequeue loop, retire.  All threads call it.
 template <class T>
 __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, char* smem,
-                                      uint32_t* s_base, uint32_t* s_total) {
-  const uint32_t flags = d->flags;
-  const uint32_t chunk = d->chunk;
+                                      uint32_t* s_base, uint32_t* s_total, uint32_t cfg) {
+  const uint32_t chunk = cfg & kCfgChunkMask;
+  const bool resolve = (cfg & kCfgResolve) != 0;
+  const bool depth2 = !resolve && (cfg & kCfgDepth2) != 0;
+  const bool stride = !resolve && (cfg & kCfgStride) != 0;
+  bool admitted = true;  // meaningful in thread 0 only
+  uint32_t p1 = kTerminate;  // thread 0: dequeue issued one iteration earlier (depth 2)
+  uint32_t iter = 0;         // stride mode: iteration count
+  if (threadIdx.x == 0) {  // master work-item: environment init (rt_env_init)
+    uint32_t b = kTerminate;
+    // STATIC: the first dequeue is issued before anything else is loaded
+    if (stride) b = blockIdx.x * chunk;
+    else if (!resolve) b = atomicAdd(&d->next, chunk);
+    if (depth2) p1 = atomicAdd(&d->next, chunk);
+    if (cfg & kCfgStamps) red_min_u64(&d->t_first, globaltimer());
+    const uint32_t total = vg_total<T>(args, d, d->launch_idx);
+    if (blockIdx.x == 0 || resolve) d->total_seen = total;
+    if (resolve) {
+      atomicMax(&d->ctl->cur, d->req_idx);
+      admitted = admit(d);
+      if (admitted) b = dequeue(d, chunk, true, admitted);
+    }
+    if (b < total) red_add_u32(&d->ctas_started, 1u);
+    *s_total = total;
+    s_base[0] = b;
+  }
   const uint32_t launch_idx = d->launch_idx;
   const uint32_t gx = d->gx, gy = d->gy, gz = d->gz;
   uint32_t* const coverage = d->coverage;
-  bool admitted = false;  // meaningful in thread 0 only
-  if (threadIdx.x == 0) {  // master work-item: environment init (rt_env_init)
-    if (flags & kFlagStamps) atomicMin(&d->t_first, globaltimer());
-    if (d->ctl != nullptr) atomicMax(&d->ctl->cur, d->req_idx);
-    const uint32_t total = vg_total<T>(args, d, launch_idx);
-    *s_total = total;
-    if (d->total_seen != total) d->total_seen = total;
-    admitted = admit(d, flags);
-    uint32_t b = kTerminate;
-    if (admitted) {
-      b = dequeue(d, chunk, admitted);
-      if (b < total) atomicAdd(&d->ctas_started, 1u);
-    }
-    s_base[0] = b;
-  }
   __syncthreads();
   const uint32_t total = *s_total;
   uint32_t buf = 0;
@@ -232,7 +266,10 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     const uint32_t base = s_base[buf];
     if (base >= total) break;                  // RUN_TERMINATE
     uint32_t nxt = 0;
-    if (threadIdx.x == 0) nxt = dequeue(d, chunk, admitted);  // prefetch next chunk
+    if (threadIdx.x == 0) {                    // prefetch the next chunk id
+      if (stride) nxt = (blockIdx.x + (++iter) * gridDim.x) * chunk;
+      else nxt = dequeue(d, chunk, resolve, admitted);
+    }
     const uint32_t end = min(base + chunk, total);
     for (uint32_t vg = base; vg < end; ++vg) {
       const VirtualBlock vb = decode(vg, gx, gy, gz, launch_idx);
@@ -240,25 +277,34 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
       if (coverage != nullptr && threadIdx.x == 0) atomicAdd(&coverage[vg], 1u);
       if (vg + 1 < end) __syncthreads();       // body smem reuse across VGs
     }
-    if (threadIdx.x == 0) s_base[buf ^ 1] = nxt;
+    if (threadIdx.x == 0) {
+      if (depth2) {  // publish the id requested one iteration ago
+        s_base[buf ^ 1] = p1;
+        p1 = nxt;
+      } else {
+        s_base[buf ^ 1] = nxt;
+      }
+    }
     __syncthreads();
     buf ^= 1;
   }
-  if (threadIdx.x == 0) retire(d, flags, admitted);
+  if (threadIdx.x == 0) retire(d, cfg, admitted);
 }
 
 // -------------------------------------------------------------------------
 // The scheduling kernel: grid = quota (1-D), block = the original block;
-// serves launch d.
+// serves launch d.  cfg = chunk | kCfg* flags.
 template <class T>
 __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
-    accel_persistent(const typename T::Args args, Desc* __restrict__ d, uint32_t /*unused*/) {
+    accel_persistent(const typename T::Args args, Desc* __restrict__ d, uint32_t cfg) {
   extern __shared__ __align__(128) char smem[];
   __shared__ uint32_t s_base[2];   // double-buffered dequeue result (sd.wg_base)
   __shared__ uint32_t s_total;
-  if (threadIdx.x == 0 && d->has_prev && ld_volatile(&(d - 1)->topped)) wait_complete(d - 1);
-  __syncthreads();
-  serve<T>(args, d, smem, s_base, &s_total);
+  if (cfg & kCfgResolve) {
+    if (threadIdx.x == 0 && d->has_prev && ld_volatile(&(d - 1)->topped)) wait_complete(d - 1);
+    __syncthreads();
+  }
+  serve<T>(args, d, smem, s_base, &s_total, cfg);
 }
 
 // RESOLVE top-up grid: d = first launch of the request step, `sticky` =
@@ -284,7 +330,8 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
       __threadfence();
     }
     __syncthreads();
-    serve<T>(args, dl, smem, s_base, &s_total);
+    const uint32_t cfg = dl->chunk | kCfgResolve | ((dl->flags & kFlagStamps) ? kCfgStamps : 0u);
+    serve<T>(args, dl, smem, s_base, &s_total, cfg);
     __syncthreads();
   }
 }
@@ -295,7 +342,7 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
     accel_native(const typename T::Args args, Desc* __restrict__ d, uint32_t /*unused*/) {
   extern __shared__ __align__(128) char smem[];
   const uint32_t flags = d->flags;
-  if (threadIdx.x == 0 && (flags & kFlagStamps)) atomicMin(&d->t_first, globaltimer());
+  if (threadIdx.x == 0 && (flags & kFlagStamps)) red_min_u64(&d->t_first, globaltimer());
   VirtualBlock vb;
   vb.x = blockIdx.x; vb.y = blockIdx.y; vb.z = blockIdx.z;
   vb.gx = gridDim.x; vb.gy = gridDim.y; vb.gz = gridDim.z;
@@ -312,7 +359,7 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
     T::body(args, vb, smem);
     if (d->coverage != nullptr && threadIdx.x == 0) atomicAdd(&d->coverage[vb.linear], 1u);
   }
-  if (threadIdx.x == 0 && (flags & kFlagStamps)) atomicMax(&d->t_last, globaltimer());
+  if (threadIdx.x == 0 && (flags & kFlagStamps)) red_max_u64(&d->t_last, globaltimer());
 }
 
 }  // namespace accel

@@ -34,7 +34,7 @@ struct InitParams {
 cudaError_t launch_desc_init(const InitParams& p, uint32_t n_desc, cudaStream_t s);
 // RESOLVE: wait (1 thread) until the request's last launch and its top-ups completed.
 cudaError_t launch_join(const Desc* last, cudaStream_t s);
-constexpr size_t kDescBytes = 256;
+constexpr size_t kDescBytes = 384;
 constexpr size_t kCtlBytes = 16;
 
 }  // namespace accel

@@ -109,11 +109,17 @@ std::string g_init_error;
 
 // Host view of the device descriptor (csrc/device/dispatch.cuh accel::Desc).
 struct DescHost {
-  uint32_t total, gx, gy, gz, chunk, launch_idx, flags, total_seen;
-  uint64_t live_quota, coverage;
+  // line 0
+  uint32_t total, gx, gy, gz, chunk, launch_idx, flags, req_idx;
+  uint64_t ctl, coverage;
+  uint32_t has_prev, pad0[19];
+  // line 1
+  uint32_t next, pad1[31];
+  // line 2
   unsigned long long t_first, t_last;
-  uint32_t ctas_started, alive, max_alive, topped, req_idx, has_prev;
+  uint32_t total_seen, ctas_started, alive, max_alive, topped, pad2[23];
 };
+static_assert(sizeof(DescHost) == accel::kDescBytes, "host view of the descriptor");
 
 }  // namespace
 
@@ -141,6 +147,9 @@ struct accel_ctx {
   std::thread monitor;
   std::atomic<bool> stop{false};
   uint64_t monitor_solves = 0;
+  // dispatch variant (env ACCEL_DISPATCH): "" / "dyn" = one dequeue in flight,
+  // "dyn2" = two in flight (kCfgDepth2), "stride" = static round robin (ablation)
+  uint32_t dispatch_bits = 0;
   std::vector<uint8_t> slot_used;
   std::map<uint64_t, std::unique_ptr<Request>> reqs;
   uint64_t next_id = 1;
@@ -278,8 +287,9 @@ int enqueue(accel_ctx* ctx, Request* r) {
     for (uint32_t l = 0; l < st.repeat; ++l, ++li) {
       if (lev) CK(ctx, cudaEventRecord(r->ev_launch[li], s));
       accel::Desc* d = ctx->desc_ptr(r->slot + st.first + l);
-      uint32_t sticky = 0;
-      void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &sticky};
+      // accel_persistent cfg word (dispatch.cuh): chunk | kCfgResolve | kCfgStamps
+      uint32_t cfg = (k.chunk & 0xffffu) | (resolve ? (1u << 16) : 0u) | (1u << 17) | ctx->dispatch_bits;
+      void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &cfg};
       const dim3 grid = shared ? dim3(st.quota, 1, 1) : dim3(st.grid.x, st.grid.y, st.grid.z);
       CK(ctx, cudaLaunchKernel(shared ? k.pfn : k.nfn, grid, k.block, params, k.dyn_smem, s));
     }
@@ -536,6 +546,10 @@ int accel_init(const accel_config* cfg, accel_ctx** out) {
                          cudaHostAllocDefault)) != cudaSuccess)
     return init_fail(e, "cudaHostAlloc(ring)");
   ctx->slot_used.assign(kPoolSlots, 0);
+  if (const char* dv = std::getenv("ACCEL_DISPATCH")) {
+    if (std::strcmp(dv, "dyn2") == 0) ctx->dispatch_bits = 1u << 18;
+    if (std::strcmp(dv, "stride") == 0) ctx->dispatch_bits = 1u << 19;
+  }
   accel_ctx* raw = ctx.release();
   raw->monitor = std::thread(monitor_loop, raw);
   *out = raw;

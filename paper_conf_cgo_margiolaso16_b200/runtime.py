@@ -17,13 +17,19 @@ from .jobs import Job  # noqa: E402
 
 class Accel:
     def __init__(self, device: int = 0, mode: int = abi.MODE_SHARED, policy: int = abi.POLICY_STATIC,
-                 verify: bool = False, caps: abi.accel_caps | None = None):
+                 verify: bool = False, caps: abi.accel_caps | None = None,
+                 chunks: dict[str, int] | None = None):
+        """chunks: per-kernel override of the VGs taken per dequeue (PAPER.md
+        §6.4 adaptive scheduling; 1 = the paper's "naive" variant)."""
         self.device = device
         self.ctx = abi.accel_init(device, mode, policy, verify, caps)
         self.mode, self.policy, self.verify = mode, policy, verify
         self.kids: dict[str, int] = {}
         for name in abi.accel_builtin_names():
-            self.kids[name] = abi.accel_kernel_register(self.ctx, abi.accel_builtin_kernel(name))
+            desc = abi.accel_builtin_kernel(name)
+            if chunks and name in chunks:
+                desc.chunk = chunks[name]
+            self.kids[name] = abi.accel_kernel_register(self.ctx, desc)
 
     def close(self):
         if self.ctx:

@@ -25,9 +25,11 @@ def main():
     ap.add_argument("tenants", nargs="+")
     ap.add_argument("--size", default="default")
     ap.add_argument("--reps", type=int, default=5)
-    ap.add_argument("--chunk1", action="store_true")
+    ap.add_argument("--chunk", type=int, default=0, help="override VGs per dequeue for all kernels")
     args = ap.parse_args()
-    acc = Accel(0)
+    from paper_conf_cgo_margiolaso16_b200 import abi as _abi
+    chunks = {n: args.chunk for n in _abi.accel_builtin_names()} if args.chunk else None
+    acc = Accel(0, chunks=chunks)
     flush = torch.empty(64 * 1024 * 1024, dtype=torch.float32, device="cuda")
     out = {}
     for t in args.tenants:
