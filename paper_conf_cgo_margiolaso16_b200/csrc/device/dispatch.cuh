@@ -78,7 +78,10 @@ struct alignas(128) Desc {
   uint32_t alive;        // CTAs currently admitted (RESOLVE)
   uint32_t max_alive;    // high-water mark of `alive` (RESOLVE)
   uint32_t topped;       // a top-up CTA joined this launch (RESOLVE)
-  uint32_t pad2[23];
+  uint32_t admit_fail;   // RESOLVE: CTAs refused at admission
+  uint32_t evicted;      // RESOLVE: CTAs that left at a dequeue (shrink)
+  uint32_t last_live;    // RESOLVE: live quota seen by the last refused CTA
+  uint32_t pad2[20];
 };
 static_assert(sizeof(Desc) == 384, "Desc layout");
 
@@ -192,28 +195,42 @@ enum : uint32_t {
 // Master work-item, admission into launch d under RESOLVE (count-based):
 // returns false if the launch already holds `live` CTAs.
 __device__ __forceinline__ bool admit(Desc* d) {
-  const uint32_t a = atomicAdd(&d->alive, 1u) + 1u;
-  if (a > ld_volatile(&d->ctl->live)) {
-    atomicSub(&d->alive, 1u);
-    return false;
+  // compare-and-swap, so a refused CTA never inflates `alive` (an atomicAdd
+  // followed by an atomicSub would make admitted CTAs see a transient
+  // alive > live and evict themselves)
+  const uint32_t live = ld_volatile(&d->ctl->live);
+  uint32_t a = ld_volatile(&d->alive);
+  for (;;) {
+    if (a >= live) {
+      red_add_u32(&d->admit_fail, 1u);
+      d->last_live = live;
+      return false;
+    }
+    const uint32_t prev = atomicCAS(&d->alive, a, a + 1u);
+    if (prev == a) break;
+    a = prev;
   }
-  atomicMax(&d->max_alive, a);
+  atomicMax(&d->max_alive, a + 1u);
   __threadfence();  // admission visible before the first dequeue
   return true;
 }
 
 // One dequeue (Fig. 8b line 26, rt_sched_wgroup): under RESOLVE a CTA
 // leaves first if the launch holds more CTAs than the live quota (shrink at a
-// VG boundary); then one atomicAdd of `chunk` on the queue head.
+// VG boundary; CAS so exactly alive - live CTAs leave); then one atomicAdd of
+// `chunk` on the queue head.
 __device__ __forceinline__ uint32_t dequeue(Desc* d, uint32_t chunk, bool resolve, bool& admitted) {
   if (resolve) {
     const uint32_t live = ld_volatile(&d->ctl->live);
-    if (ld_volatile(&d->alive) > live) {
-      if (atomicSub(&d->alive, 1u) > live) {
+    uint32_t a = ld_volatile(&d->alive);
+    while (a > live) {
+      const uint32_t prev = atomicCAS(&d->alive, a, a - 1u);
+      if (prev == a) {
+        red_add_u32(&d->evicted, 1u);
         admitted = false;
         return kTerminate;
       }
-      atomicAdd(&d->alive, 1u);
+      a = prev;
     }
   }
   return atomicAdd(&d->next, chunk);

@@ -74,6 +74,9 @@ struct Request {
   std::vector<accel_copy> h2d, d2h;
   cudaEvent_t ev_arrival = nullptr, ev_done = nullptr;
   std::vector<cudaEvent_t> ev_launch;  // ACCEL_REQ_LAUNCH_EVENTS: n_desc + 1
+  // RESOLVE: one event after every top-up grid.  The request's descriptors
+  // may only be released (and reused) once its sticky top-up CTAs retired.
+  std::vector<cudaEvent_t> ev_topups;
   uint32_t slot = 0, n_desc = 0;
   uint32_t* cov = nullptr;
   uint64_t cov_elems = 0;
@@ -117,7 +120,7 @@ struct DescHost {
   uint32_t next, pad1[31];
   // line 2
   unsigned long long t_first, t_last;
-  uint32_t total_seen, ctas_started, alive, max_alive, topped, pad2[23];
+  uint32_t total_seen, ctas_started, alive, max_alive, topped, admit_fail, evicted, last_live, pad2[20];
 };
 static_assert(sizeof(DescHost) == accel::kDescBytes, "host view of the descriptor");
 
@@ -199,9 +202,12 @@ struct accel_ctx {
 
 namespace {
 
+bool debug_on();
+
 int refresh_done(accel_ctx* ctx, Request* r) {
   if (r->done) return ACCEL_OK;
   cudaError_t e = cudaEventQuery(r->ev_done);
+  for (size_t i = 0; e == cudaSuccess && i < r->ev_topups.size(); ++i) e = cudaEventQuery(r->ev_topups[i]);
   if (e == cudaSuccess) {
     r->done = true;
   } else if (e != cudaErrorNotReady) {
@@ -241,9 +247,24 @@ int fetch_result(accel_ctx* ctx, Request* r) {
         // dynamic-total kernels (bfs) cover only the live part of the static grid
         const uint32_t live = d->total_seen <= s.total ? d->total_seen : s.total;
         const uint32_t* c = cov.data() + s.cov_offset + (uint64_t)l * s.total;
+        uint32_t bad = 0, first_bad = 0, got = 0;
         for (uint32_t v = 0; v < s.total; ++v) {
           const uint32_t want = v < live ? 1u : 0u;
-          if (c[v] != want) ok = false;
+          if (c[v] != want) {
+            if (bad++ == 0) {
+              first_bad = v;
+              got = c[v];
+            }
+          }
+        }
+        if (bad) {
+          ok = false;
+          if (debug_on())
+            std::fprintf(stderr,
+                         "[accel] coverage: req %llu tenant %d launch %u: %u bad VGs (first %u ran %u times), "
+                         "total %u seen %u next %u topped %u alive %u refused %u evicted %u live %u\n",
+                         (unsigned long long)r->id, r->tenant, s.first + l, bad, first_bad, got, s.total,
+                         d->total_seen, d->next, d->topped, d->alive, d->admit_fail, d->evicted, d->last_live);
         }
       }
     r->cov_ok = ok ? 1 : 0;
@@ -360,6 +381,7 @@ int apply_quota(accel_ctx* ctx, Request* r, uint32_t q) {
     std::fprintf(stderr, "[accel] resolve req %llu tenant %d live %u -> %u (provisioned %u)\n",
                  (unsigned long long)r->id, r->tenant, r->live, q, r->provisioned);
   if (q == r->live) return ACCEL_OK;
+  if (cudaEventQuery(r->ev_done) == cudaSuccess) return ACCEL_OK;  // finished: nothing to grow
   uint32_t* h = ctx->pinned_ring + (ctx->ring_pos++ % kRing);
   *h = q;
   CK(ctx, cudaMemcpyAsync(ctx->ctl_pool + (size_t)r->slot * kCtlBytes /* Ctl::live */, h, sizeof(uint32_t), cudaMemcpyHostToDevice, ctx->ctl));
@@ -369,8 +391,12 @@ int apply_quota(accel_ctx* ctx, Request* r, uint32_t q) {
     accel::Desc* d = ctx->desc_ptr(r->slot + st.first);
     uint32_t sticky = st.repeat;
     void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &sticky};
-    CK(ctx, cudaLaunchKernel(k.tfn, dim3(q - r->provisioned, 1, 1), k.block, params, k.dyn_smem,
-                             ctx->topup[ctx->topup_rr++ % accel_ctx::kTopupStreams]));
+    cudaStream_t ts = ctx->topup[ctx->topup_rr++ % accel_ctx::kTopupStreams];
+    CK(ctx, cudaLaunchKernel(k.tfn, dim3(q - r->provisioned, 1, 1), k.block, params, k.dyn_smem, ts));
+    cudaEvent_t ev;
+    CK(ctx, ctx->get_event(&ev));
+    r->ev_topups.push_back(ev);
+    CK(ctx, cudaEventRecord(ev, ts));
     r->provisioned = q;
   }
   r->live = q;
@@ -502,6 +528,7 @@ void release_request(accel_ctx* ctx, Request* r) {
   if (r->ev_arrival) ctx->free_events.push_back(r->ev_arrival);
   if (r->ev_done) ctx->free_events.push_back(r->ev_done);
   for (cudaEvent_t ev : r->ev_launch) ctx->free_events.push_back(ev);
+  for (cudaEvent_t ev : r->ev_topups) ctx->free_events.push_back(ev);
 }
 
 }  // namespace
@@ -563,6 +590,7 @@ int accel_finalize(accel_ctx* ctx) {
   cudaSetDevice(ctx->cfg.device);
   for (auto& kv : ctx->reqs) {
     if (kv.second->ev_done) cudaEventSynchronize(kv.second->ev_done);
+    for (cudaEvent_t ev : kv.second->ev_topups) cudaEventSynchronize(ev);
     release_request(ctx, kv.second.get());
   }
   ctx->reqs.clear();
@@ -664,35 +692,51 @@ int accel_submit(accel_ctx* ctx, const accel_request* r, uint64_t* id) {
 
 int accel_sync(accel_ctx* ctx, uint64_t request_id) {
   if (!ctx) return ACCEL_EINVAL;
-  std::vector<std::pair<uint64_t, cudaEvent_t>> wait;
-  {
-    std::lock_guard<std::mutex> g(ctx->mu);
-    if (ctx->poisoned) return ACCEL_ESTATE;
-    CK(ctx, cudaSetDevice(ctx->cfg.device));
-    if (request_id == ACCEL_ALL) {
-      for (auto& kv : ctx->reqs) wait.emplace_back(kv.first, kv.second->ev_done);
-    } else {
-      auto it = ctx->reqs.find(request_id);
-      if (it == ctx->reqs.end()) return ctx->fail(ACCEL_EINVAL, "unknown request");
-      wait.emplace_back(request_id, it->second->ev_done);
-    }
-  }
-  // wait without the lock: the RESOLVE monitor keeps re-solving meanwhile
-  for (auto& w : wait) {
-    cudaError_t e = cudaEventSynchronize(w.second);
-    if (e != cudaSuccess) {
+  std::vector<uint64_t> ids;
+  // Wait without holding the lock (the RESOLVE monitor keeps re-solving
+  // meanwhile); it may add top-up grids to a request while we wait, so repeat
+  // until every event of every request is complete.
+  for (;;) {
+    std::vector<cudaEvent_t> wait;
+    {
       std::lock_guard<std::mutex> g(ctx->mu);
-      return ctx->cuda(e, "cudaEventSynchronize");
+      if (ctx->poisoned) return ACCEL_ESTATE;
+      CK(ctx, cudaSetDevice(ctx->cfg.device));
+      ids.clear();
+      if (request_id == ACCEL_ALL) {
+        for (auto& kv : ctx->reqs) ids.push_back(kv.first);
+      } else {
+        if (ctx->reqs.find(request_id) == ctx->reqs.end()) return ctx->fail(ACCEL_EINVAL, "unknown request");
+        ids.push_back(request_id);
+      }
+      for (uint64_t id : ids) {
+        Request* r = ctx->reqs[id].get();
+        int rc = refresh_done(ctx, r);
+        if (rc) return rc;
+        if (r->done) continue;
+        wait.push_back(r->ev_done);
+        for (cudaEvent_t ev : r->ev_topups) wait.push_back(ev);
+      }
+    }
+    if (wait.empty()) break;
+    for (cudaEvent_t ev : wait) {
+      cudaError_t e = cudaEventSynchronize(ev);
+      if (e != cudaSuccess) {
+        std::lock_guard<std::mutex> g(ctx->mu);
+        return ctx->cuda(e, "cudaEventSynchronize");
+      }
     }
   }
   std::lock_guard<std::mutex> g(ctx->mu);
   bool cov_bad = false;
-  for (auto& w : wait) {
-    auto it = ctx->reqs.find(w.first);
+  for (uint64_t id : ids) {
+    auto it = ctx->reqs.find(id);
     if (it == ctx->reqs.end()) continue;
     Request* r = it->second.get();
-    r->done = true;
-    int rc = fetch_result(ctx, r);
+    int rc = refresh_done(ctx, r);
+    if (rc) return rc;
+    if (!r->done) return ctx->fail(ACCEL_ESTATE, "request not complete after sync");
+    rc = fetch_result(ctx, r);
     if (rc) return rc;
     if (r->cov_ok == 0) cov_bad = true;
   }
