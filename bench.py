@@ -229,6 +229,37 @@ def run_reference(args):
     print(json.dumps(line), flush=True)
 
 
+def aggregate(allres: list[dict], world: int, steps: int, policy: str) -> dict:
+    """Whole-job figures from the per-rank results: device times are the max
+    over ranks (the job ends when the slowest GPU ends); value = all mixes
+    completed on all GPUs / that time (weak scaling: each GPU runs its own
+    mix); sharing metrics are geometric (U) / arithmetic (STP, ANTT) means
+    over every rank's steps."""
+    gm = lambda xs: math.exp(statistics.mean(math.log(x) for x in xs))  # noqa: E731
+    tmax = max(r["dev_ms"] for r in allres)
+    emax = max(r["e2e_ms"] for r in allres)
+    nmax = max(r["nat_ms"] for r in allres)
+    omax = max(r["oth_ms"] for r in allres)
+    return {
+        "tmax": tmax, "emax": emax, "nmax": nmax,
+        "value": world * steps / (tmax / 1e3),
+        "U_sh": gm([u for r in allres for u in r["sh"]["U"]]),
+        "U_na": gm([u for r in allres for u in r["na"]["U"]]),
+        "stp_sh": statistics.mean(u for r in allres for u in r["sh"]["STP"]),
+        "stp_na": statistics.mean(u for r in allres for u in r["na"]["STP"]),
+        "antt_sh": statistics.mean(u for r in allres for u in r["sh"]["ANTT"]),
+        "antt_na": statistics.mean(u for r in allres for u in r["na"]["ANTT"]),
+        "other": {
+            "policy": "static" if policy == "resolve" else "resolve",
+            "unfairness": gm([u for r in allres for u in r["ot"]["U"]]),
+            "stp": statistics.mean(u for r in allres for u in r["ot"]["STP"]),
+            "antt": statistics.mean(u for r in allres for u in r["ot"]["ANTT"]),
+            "mixes_per_s": world * steps / (omax / 1e3),
+            "throughput_speedup": nmax / omax,
+        },
+    }
+
+
 # ----------------------------------------------------------------- GPU leg
 def main():
     ap = argparse.ArgumentParser()
@@ -401,28 +432,11 @@ def main():
                                 "on all host cores)"}
 
     if rank == 0:
-        tmax = max(r["dev_ms"] for r in allres)
-        emax = max(r["e2e_ms"] for r in allres)
-        nmax = max(r["nat_ms"] for r in allres)
-        value = world * args.steps / (tmax / 1e3)
-        gm = lambda xs: math.exp(statistics.mean(math.log(x) for x in xs))  # noqa: E731
-        U_sh = gm([u for r in allres for u in r["sh"]["U"]])
-        U_na = gm([u for r in allres for u in r["na"]["U"]])
-        stp_sh = statistics.mean(u for r in allres for u in r["sh"]["STP"])
-        stp_na = statistics.mean(u for r in allres for u in r["na"]["STP"])
-        antt_sh = statistics.mean(u for r in allres for u in r["sh"]["ANTT"])
-        antt_na = statistics.mean(u for r in allres for u in r["na"]["ANTT"])
-        omax = max(r["oth_ms"] for r in allres)
-        other_name = "static" if args.policy == "resolve" else "resolve"
-        other_sum = {
-            "policy": other_name,
-            "unfairness": gm([u for r in allres for u in r["ot"]["U"]]),
-            "stp": statistics.mean(u for r in allres for u in r["ot"]["STP"]),
-            "antt": statistics.mean(u for r in allres for u in r["ot"]["ANTT"]),
-            "mixes_per_s": world * args.steps / (omax / 1e3),
-            "throughput_speedup": nmax / omax,
-            "T_s_ms": dict(zip(tenants, np.mean(allres[0]["ot"]["ts_ms"], 0).tolist())),
-        }
+        agg = aggregate(allres, world, args.steps, args.policy)
+        tmax, emax, nmax, value = agg["tmax"], agg["emax"], agg["nmax"], agg["value"]
+        U_sh, U_na, stp_sh, stp_na = agg["U_sh"], agg["U_na"], agg["stp_sh"], agg["stp_na"]
+        antt_sh, antt_na, other_sum = agg["antt_sh"], agg["antt_na"], agg["other"]
+        other_sum["T_s_ms"] = dict(zip(tenants, np.mean(allres[0]["ot"]["ts_ms"], 0).tolist()))
         clocks = allres[0]["clk"]
         line = {
             "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": args.steps,
@@ -451,7 +465,7 @@ def main():
             },
             "e2e": {"value": world * args.steps / (emax / 1e3), "unit": UNIT,
                     "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h},
-            "gpu_launches": launches_per_step * args.steps,
+            "gpu_launches": launches_per_step * args.steps * world,
             "roofline": dict(roof[dom], kernel=dom) if dom else None,
             "rooflines": roof,
             "cpu_baseline": cpu,
