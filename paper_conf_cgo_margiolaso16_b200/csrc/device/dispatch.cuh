@@ -180,15 +180,12 @@ __device__ __forceinline__ void wait_complete(const Desc* p) {
 
 // Launch configuration word, a kernel parameter (no descriptor load on the
 // critical path of a CTA's first dequeue): bits 0-15 chunk, then flags.
-//   kCfgDepth2: two dequeues in flight per CTA (the next VG id is requested
-//               two VGs ahead, hiding atomic latency behind long VG bodies).
 //   kCfgStride: static round-robin VG assignment (VG = cta + i * grid), no
 //               queue -- an ablation to measure the cost of the dynamic queue.
 enum : uint32_t {
   kCfgChunkMask = 0xffffu,
   kCfgResolve = 1u << 16,
   kCfgStamps = 1u << 17,
-  kCfgDepth2 = 1u << 18,
   kCfgStride = 1u << 19
 };
 
@@ -244,25 +241,35 @@ __device__ __forceinline__ void retire(Desc* d, uint32_t cfg, bool admitted) {
   if (cfg & kCfgStamps) red_max_u64(&d->t_last, globaltimer());
 }
 
+// Scheduling state of one CTA in shared memory (the paper's `local struct SD`,
+// Fig. 8b).  Keeping it in shared memory instead of registers
+// leaves the body the same register budget it has in the native kernel: only
+// the current VG id and the prefetched chunk id live across the body call.
+struct SchedState {
+  uint32_t cur;        // VG to run next (sd.wg_base)
+  uint32_t end;        // end of the current chunk (sd.wg_end)
+  uint32_t total;      // VGs of this launch (RUN_TERMINATE when cur >= total)
+  uint32_t gx, gy, gz, launch_idx;
+  uint32_t* coverage;
+};
+
 // Serve one launch: admission, dequeue loop, retire.  All threads call it.
 template <class T>
 __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, char* smem,
-                                      uint32_t* s_base, uint32_t* s_total, uint32_t cfg) {
+                                      SchedState* S, uint32_t cfg) {
   const uint32_t chunk = cfg & kCfgChunkMask;
   const bool resolve = (cfg & kCfgResolve) != 0;
-  const bool depth2 = !resolve && (cfg & kCfgDepth2) != 0;
   const bool stride = !resolve && (cfg & kCfgStride) != 0;
-  bool admitted = true;  // meaningful in thread 0 only
-  uint32_t p1 = kTerminate;  // thread 0: dequeue issued one iteration earlier (depth 2)
-  uint32_t iter = 0;         // stride mode: iteration count
-  if (threadIdx.x == 0) {  // master work-item: environment init (rt_env_init)
+  bool admitted = true;      // meaningful in thread 0 only
+  uint32_t iter = 0;         // stride ablation: chunks taken so far (thread 0)
+  if (threadIdx.x == 0) {    // master work-item: environment init (rt_env_init)
     uint32_t b = kTerminate;
     // STATIC: the first dequeue is issued before anything else is loaded
     if (stride) b = blockIdx.x * chunk;
     else if (!resolve) b = atomicAdd(&d->next, chunk);
-    if (depth2) p1 = atomicAdd(&d->next, chunk);
     if (cfg & kCfgStamps) red_min_u64(&d->t_first, globaltimer());
-    const uint32_t total = vg_total<T>(args, d, d->launch_idx);
+    const uint32_t launch_idx = d->launch_idx;
+    const uint32_t total = vg_total<T>(args, d, launch_idx);
     if (blockIdx.x == 0 || resolve) d->total_seen = total;
     if (resolve) {
       atomicMax(&d->ctl->cur, d->req_idx);
@@ -270,40 +277,39 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
       if (admitted) b = dequeue(d, chunk, true, admitted);
     }
     if (b < total) red_add_u32(&d->ctas_started, 1u);
-    *s_total = total;
-    s_base[0] = b;
+    S->cur = b;
+    S->end = b < total ? min(b + chunk, total) : b;
+    S->total = total;
+    S->gx = d->gx;
+    S->gy = d->gy;
+    S->gz = d->gz;
+    S->launch_idx = launch_idx;
+    S->coverage = d->coverage;
   }
-  const uint32_t launch_idx = d->launch_idx;
-  const uint32_t gx = d->gx, gy = d->gy, gz = d->gz;
-  uint32_t* const coverage = d->coverage;
   __syncthreads();
-  const uint32_t total = *s_total;
-  uint32_t buf = 0;
+  uint32_t nxt = kTerminate;  // thread 0: id of the next chunk, requested at chunk start
+  bool have_nxt = false;
   for (;;) {
-    const uint32_t base = s_base[buf];
-    if (base >= total) break;                  // RUN_TERMINATE
-    uint32_t nxt = 0;
-    if (threadIdx.x == 0) {                    // prefetch the next chunk id
+    const uint32_t vg = S->cur;
+    if (vg >= S->total) break;                 // RUN_TERMINATE
+    if (threadIdx.x == 0 && !have_nxt) {
+      // prefetch the next chunk id once per chunk, early (hidden behind the body)
       if (stride) nxt = (blockIdx.x + (++iter) * gridDim.x) * chunk;
       else nxt = dequeue(d, chunk, resolve, admitted);
+      have_nxt = true;
     }
-    const uint32_t end = min(base + chunk, total);
-    for (uint32_t vg = base; vg < end; ++vg) {
-      const VirtualBlock vb = decode(vg, gx, gy, gz, launch_idx);
-      T::body(args, vb, smem);
-      if (coverage != nullptr && threadIdx.x == 0) atomicAdd(&coverage[vg], 1u);
-      if (vg + 1 < end) __syncthreads();       // body smem reuse across VGs
-    }
+    T::body(args, decode(vg, S->gx, S->gy, S->gz, S->launch_idx), smem);
     if (threadIdx.x == 0) {
-      if (depth2) {  // publish the id requested one iteration ago
-        s_base[buf ^ 1] = p1;
-        p1 = nxt;
-      } else {
-        s_base[buf ^ 1] = nxt;
+      if (S->coverage != nullptr) atomicAdd(&S->coverage[vg], 1u);
+      if (vg + 1 < S->end) {
+        S->cur = vg + 1;
+      } else {                                   // publish the prefetched chunk
+        S->cur = nxt;
+        S->end = nxt < S->total ? min(nxt + chunk, S->total) : nxt;
+        have_nxt = false;
       }
     }
     __syncthreads();
-    buf ^= 1;
   }
   if (threadIdx.x == 0) retire(d, cfg, admitted);
 }
@@ -315,13 +321,12 @@ template <class T>
 __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
     accel_persistent(const typename T::Args args, Desc* __restrict__ d, uint32_t cfg) {
   extern __shared__ __align__(128) char smem[];
-  __shared__ uint32_t s_base[2];   // double-buffered dequeue result (sd.wg_base)
-  __shared__ uint32_t s_total;
+  __shared__ SchedState S;
   if (cfg & kCfgResolve) {
     if (threadIdx.x == 0 && d->has_prev && ld_volatile(&(d - 1)->topped)) wait_complete(d - 1);
     __syncthreads();
   }
-  serve<T>(args, d, smem, s_base, &s_total, cfg);
+  serve<T>(args, d, smem, &S, cfg);
 }
 
 // RESOLVE top-up grid: d = first launch of the request step, `sticky` =
@@ -331,8 +336,7 @@ template <class T>
 __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
     accel_topup(const typename T::Args args, Desc* __restrict__ d, uint32_t sticky) {
   extern __shared__ __align__(128) char smem[];
-  __shared__ uint32_t s_base[2];
-  __shared__ uint32_t s_total;
+  __shared__ SchedState S;
   __shared__ uint32_t s_l;
   if (threadIdx.x == 0) {
     const uint32_t cur = ld_volatile(&d->ctl->cur);
@@ -348,7 +352,7 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
     }
     __syncthreads();
     const uint32_t cfg = dl->chunk | kCfgResolve | ((dl->flags & kFlagStamps) ? kCfgStamps : 0u);
-    serve<T>(args, dl, smem, s_base, &s_total, cfg);
+    serve<T>(args, dl, smem, &S, cfg);
     __syncthreads();
   }
 }
