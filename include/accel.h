@@ -155,6 +155,10 @@ typedef struct {
   int32_t tenant;             /* 0..ACCEL_MAX_TENANTS-1: selects the stream pair */
   uint32_t flags;             /* ACCEL_REQ_* */
   uint32_t weight;            /* sharing ratio (§2.2); 0 -> 1          */
+  int32_t main_step;          /* step that represents the request in the solver
+                                 (its main computation); -1 = the step with the
+                                 most virtual groups.  Every other step is solved
+                                 against the same active set with its own kernel */
   uint32_t n_steps;           /* 1..ACCEL_MAX_STEPS                             */
   const accel_launch *steps;
   uint32_t n_clear;           /* memsets before the first launch                */
@@ -234,6 +238,15 @@ typedef struct {
 } accel_mix_metrics;
 /* Sharing metrics of one mix from isolated times ta[k] and shared times ts[k]. */
 int accel_metrics(const double *ta, const double *ts, int32_t k, accel_mix_metrics *out);
+/* Encode a 2-D TMA tensor map (CUtensorMap, 128 B written to out128) for a
+ * row-major fp32 matrix: `inner` elements per row (contiguous), `outer` rows,
+ * rows row_stride_bytes apart (multiple of 16), box box_inner x box_outer,
+ * swizzle 0/32/64/128 (bytes).  Host only (uses the driver through the
+ * runtime; needs a driver, not a GPU context).  The tenant kernel reads the
+ * map from device memory the caller copies it to (64-B aligned). */
+int accel_tma_map_2d(void *out128, const void *gaddr, uint64_t inner, uint64_t outer,
+                     uint64_t row_stride_bytes, uint32_t box_inner, uint32_t box_outer, int32_t swizzle);
+
 /* Kernel execution overlap O = T(c)/T(t) of k
  * intervals [start[i], end[i]). */
 int accel_overlap(const double *start, const double *end, int32_t k, double *out);

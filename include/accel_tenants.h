@@ -121,6 +121,28 @@ typedef struct {
   uint32_t m, n, k;
 } accel_sgemm_args;
 
+/* sgemm_split -- tf32 split of an fp32 array for the 3xTF32 tensor-core GEMM:
+ * hi = round-to-nearest tf32 of src, lo = src - hi (exact).  block 256,
+ * VG = 4096 elements, grid ceil(n/4096).  16-B aligned arrays. */
+typedef struct {
+  const float *src;
+  float *hi;
+  float *lo;
+  uint64_t n;
+} accel_sgemm_split_args;
+
+/* sgemm_tc -- C[m][n] = A.B^T on tcgen05 tensor cores, 3xTF32
+ * (A_hi.B_hi + A_hi.B_lo + A_lo.B_hi, fp32 accumulation in TMEM).  tmaps =
+ * DEVICE pointer to four 128-B CUtensorMaps (A_hi, A_lo, B_hi, B_lo; each a
+ * K-major fp32 matrix, box 32 x 128 for A and 32 x 256 for B, 128-B swizzle,
+ * see accel_tma_map_2d).  block 128, VG = 128 x 256 tile of C,
+ * grid (ceil(n/256), ceil(m/128)).  k % 4 == 0. */
+typedef struct {
+  const void *tmaps;
+  float *c;
+  uint32_t m, n, k;
+} accel_sgemm_tc_args;
+
 /* mri-q ComputePhiMag: phimag = phir^2 + phii^2.  block 256, grid ceil(numk/256). */
 typedef struct {
   const float *phir;

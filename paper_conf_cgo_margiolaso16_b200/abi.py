@@ -69,7 +69,7 @@ class accel_copy(C.Structure):
 
 
 class accel_request(C.Structure):
-    _fields_ = [("tenant", i32), ("flags", u32), ("weight", u32), ("n_steps", u32), ("steps", C.POINTER(accel_launch)),
+    _fields_ = [("tenant", i32), ("flags", u32), ("weight", u32), ("main_step", i32), ("n_steps", u32), ("steps", C.POINTER(accel_launch)),
                 ("n_clear", u32), ("clear", C.POINTER(accel_clear)), ("n_h2d", u32),
                 ("h2d", C.POINTER(accel_copy)), ("n_d2h", u32), ("d2h", C.POINTER(accel_copy))]
 
@@ -132,6 +132,14 @@ class accel_sgemm_args(C.Structure):
     _fields_ = [("a", vp), ("b", vp), ("c", vp), ("m", u32), ("n", u32), ("k", u32)]
 
 
+class accel_sgemm_split_args(C.Structure):
+    _fields_ = [("src", vp), ("hi", vp), ("lo", vp), ("n", u64)]
+
+
+class accel_sgemm_tc_args(C.Structure):
+    _fields_ = [("tmaps", vp), ("c", vp), ("m", u32), ("n", u32), ("k", u32)]
+
+
 class accel_mriq_phimag_args(C.Structure):
     _fields_ = [("phir", vp), ("phii", vp), ("phimag", vp), ("numk", u32)]
 
@@ -145,7 +153,7 @@ EXPORTS = [
     "accel_init", "accel_finalize", "accel_set_mode", "accel_last_error", "accel_builtin_kernel",
     "accel_builtin_count", "accel_builtin_name", "accel_kernel_register", "accel_kernel_info_get",
     "accel_submit", "accel_submit_group", "accel_sync", "accel_epoch", "accel_stats", "accel_release",
-    "accel_tenant_stream", "accel_launch_times", "accel_launch_stats", "accel_demand_of", "accel_solve", "accel_metrics", "accel_overlap",
+    "accel_tenant_stream", "accel_launch_times", "accel_launch_stats", "accel_demand_of", "accel_solve", "accel_metrics", "accel_overlap", "accel_tma_map_2d",
 ]
 
 
@@ -184,6 +192,7 @@ def _load() -> C.CDLL:
         "accel_solve": (i32, [P(accel_caps), P(accel_demand), i32, P(u32)]),
         "accel_metrics": (i32, [P(f64), P(f64), i32, P(accel_mix_metrics)]),
         "accel_overlap": (i32, [P(f64), P(f64), i32, P(f64)]),
+        "accel_tma_map_2d": (i32, [vp, vp, u64, u64, u64, u32, u32, i32]),
     }
     for name, (res, args) in sig.items():
         fn = getattr(lib, name)
@@ -310,6 +319,13 @@ def accel_metrics(ta: list[float], ts: list[float]) -> accel_mix_metrics:
     m = accel_mix_metrics()
     check(lib.accel_metrics((f64 * k)(*ta), (f64 * k)(*ts), k, C.byref(m)))
     return m
+
+
+def accel_tma_map_2d(gaddr: int, inner: int, outer: int, row_stride_bytes: int, box_inner: int,
+                     box_outer: int, swizzle: int = 128) -> bytes:
+    out = (C.c_ubyte * 128)()
+    check(lib.accel_tma_map_2d(out, gaddr, inner, outer, row_stride_bytes, box_inner, box_outer, swizzle))
+    return bytes(out)
 
 
 def accel_overlap(start: list[float], end: list[float]) -> float:

@@ -216,15 +216,6 @@ int refresh_done(accel_ctx* ctx, Request* r) {
   return ACCEL_OK;
 }
 
-uint32_t step_quota(const accel_demand& main, uint32_t n_main, const accel_demand& st) {
-  if (st.grid_vgs == 0) return 0;
-  uint64_t m = (uint64_t)n_main * main.thr / st.thr;
-  m = std::min<uint64_t>(m, (uint64_t)n_main * main.regs / st.regs);
-  m = std::min<uint64_t>(m, (uint64_t)n_main * main.smem / st.smem);
-  m = std::min<uint64_t>(m, (uint64_t)n_main * main.cta / st.cta);
-  m = std::min<uint64_t>(m, st.grid_vgs);
-  return (uint32_t)std::max<uint64_t>(m, 1);
-}
 
 int demand_for(accel_ctx* ctx, const Step& s, uint32_t weight, accel_demand* d) {
   const Kernel& k = ctx->kernels[s.kid];
@@ -334,7 +325,8 @@ int build_request(accel_ctx* ctx, const accel_request& in, std::unique_ptr<Reque
   r->mode = ctx->cfg.mode;
   uint32_t n_desc = 0;
   uint64_t cov = 0;
-  r->main_step = 0;
+  if (in.main_step >= (int32_t)in.n_steps) return ctx->fail(ACCEL_EINVAL, "main_step out of range");
+  r->main_step = in.main_step >= 0 ? in.main_step : 0;
   for (uint32_t j = 0; j < in.n_steps; ++j) {
     const accel_launch& L = in.steps[j];
     if (L.kernel_id < 0 || L.kernel_id >= (int)ctx->kernels.size()) return ctx->fail(ACCEL_EINVAL, "bad kernel_id");
@@ -356,7 +348,7 @@ int build_request(accel_ctx* ctx, const accel_request& in, std::unique_ptr<Reque
     n_desc += L.repeat;
     cov += (uint64_t)L.repeat * s.total;
     r->steps.push_back(std::move(s));
-    if (r->steps.back().total > r->steps[r->main_step].total) r->main_step = (int)j;
+    if (in.main_step < 0 && r->steps.back().total > r->steps[r->main_step].total) r->main_step = (int)j;
   }
   r->n_desc = n_desc;
   r->cov_elems = ctx->cfg.verify ? cov : 0;
@@ -442,10 +434,15 @@ int assign_quotas(accel_ctx* ctx, std::vector<std::unique_ptr<Request>>& fresh) 
       if ((int)j == r->main_step) {
         s.quota = q[i];
       } else {
-        accel_demand dj;
-        rc = demand_for(ctx, s, r->weight, &dj);
+        // R-solver-8: a secondary step is solved against the same active set,
+        // with this request represented by the step's own kernel
+        std::vector<accel_demand> dsj = ds;
+        rc = demand_for(ctx, s, r->weight, &dsj[i]);
         if (rc) return ctx->fail(rc, "kernel does not fit on an SM");
-        s.quota = step_quota(ds[i], q[i], dj);
+        std::vector<uint32_t> qj(order.size());
+        rc = accel_solve(&ctx->caps, dsj.data(), (int32_t)dsj.size(), qj.data());
+        if (rc) return ctx->fail(rc, "accel_solve failed");
+        s.quota = qj[i];
       }
     }
     r->quota_initial = r->quota_min = r->quota_max = q[i];

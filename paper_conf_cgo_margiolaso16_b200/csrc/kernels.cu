@@ -13,6 +13,7 @@
 #include "tenants/mop.cuh"
 #include "tenants/mriq.cuh"
 #include "tenants/sgemm.cuh"
+#include "tenants/sgemm_tc.cuh"
 #include "tenants/spmv.cuh"
 #include "tenants/stencil.cuh"
 #include "tenants/tpacf.cuh"
@@ -100,6 +101,8 @@ const Builtin kBuiltins[] = {
     {"tpacf", &make_desc<Tpacf>},
     {"spmv", &make_desc<Spmv>},
     {"sgemm", &make_desc<Sgemm>},
+    {"sgemm_split", &make_desc<SgemmSplit>},
+    {"sgemm_tc", &make_desc<SgemmTc>},
     {"mriq_phimag", &make_desc<MriqPhiMag>},
     {"mriq_q", &make_desc<MriqQ>},
 };

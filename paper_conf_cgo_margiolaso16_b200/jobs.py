@@ -59,6 +59,7 @@ class Job:
         self.clears: list[tuple[torch.Tensor, int]] = []
         self._pinned_in: dict[str, torch.Tensor] = {}
         self._pinned_out: dict[str, torch.Tensor] = {}
+        self.main_step = -1  # -1: the library picks the step with the most VGs
 
     # ---- e2e: host buffers ----------------------------------------------
     def pin_host(self) -> None:
@@ -106,7 +107,7 @@ class Job:
                 h = self._pinned_out[k]
                 d2h[nd] = abi.accel_copy(h.data_ptr(), t.data_ptr(), t.numel() * t.element_size())
                 nd += 1
-        req = abi.accel_request(tenant, flags, weight, len(self.steps), steps, len(self.clears), clears,
+        req = abi.accel_request(tenant, flags, weight, self.main_step, len(self.steps), steps, len(self.clears), clears,
                                 nh, h2d, nd, d2h)
         req._keep = (steps, clears, h2d, d2h, keep)  # keep ctypes buffers alive until submit
         return req
@@ -330,6 +331,47 @@ class SgemmJob(Job):
         return {"flops": f, "flops_per_launch": f, "bound": "alu", "launches": 1}
 
 
+class SgemmTcJob(Job):
+    """sgemm on the tcgen05 tensor cores (3xTF32): steps split(A), split(B), tc."""
+
+    def __init__(self, d: dict, device="cuda"):
+        super().__init__(name="sgemm", device=torch.device(device))
+        self.m, self.n, self.k = d["m"], d["n"], d["k"]
+        if self.k % 4:
+            raise ValueError("sgemm needs k % 4 == 0 (16-B rows)")
+        self.inputs = {"a": _dev(d["a"].ravel(), self.device), "b": _dev(d["b"].ravel(), self.device)}
+        m, n, k = self.m, self.n, self.k
+        self.split = {x: torch.empty(sz, dtype=torch.float32, device=self.device)
+                      for x, sz in (("a_hi", m * k), ("a_lo", m * k), ("b_hi", n * k), ("b_lo", n * k))}
+        maps = b"".join([
+            abi.accel_tma_map_2d(self.split["a_hi"].data_ptr(), k, m, 4 * k, 32, 128),
+            abi.accel_tma_map_2d(self.split["a_lo"].data_ptr(), k, m, 4 * k, 32, 128),
+            abi.accel_tma_map_2d(self.split["b_hi"].data_ptr(), k, n, 4 * k, 32, 256),
+            abi.accel_tma_map_2d(self.split["b_lo"].data_ptr(), k, n, 4 * k, 32, 256)])
+        self.tmaps = torch.frombuffer(bytearray(maps), dtype=torch.uint8).to(self.device)
+        self.c = torch.empty(m * n, dtype=torch.float32, device=self.device)
+        self.out = {"c": self.c}
+        s = self.split
+        self.args_sa = abi.accel_sgemm_split_args(self.inputs["a"].data_ptr(), s["a_hi"].data_ptr(),
+                                                  s["a_lo"].data_ptr(), m * k)
+        self.args_sb = abi.accel_sgemm_split_args(self.inputs["b"].data_ptr(), s["b_hi"].data_ptr(),
+                                                  s["b_lo"].data_ptr(), n * k)
+        self.args_tc = abi.accel_sgemm_tc_args(self.tmaps.data_ptr(), self.c.data_ptr(), m, n, k)
+        self.main_step = 2
+        self.steps = [Step("sgemm_split", (_cdiv(m * k, 4096), 1, 1), self.args_sa, 1),
+                      Step("sgemm_split", (_cdiv(n * k, 4096), 1, 1), self.args_sb, 1),
+                      Step("sgemm_tc", (_cdiv(n, 256), _cdiv(m, 128), 1), self.args_tc, 1)]
+
+    def result(self):
+        return {"c": _np(self.c, np.float32).reshape(self.m, self.n)}
+
+    def work(self):
+        f = 2.0 * self.m * self.n * self.k
+        # roofline of the dominant (tc) launch: 3 tf32 products per algorithmic MAC
+        return {"flops": f, "flops_per_launch": f, "bound": "tensor", "launches": 3, "skip_launches": 2,
+                "mma_flops": 3 * f}
+
+
 class MriqJob(Job):
     """Two steps, like Parboil's mri-q: ComputePhiMag (tiny) then ComputeQ."""
 
@@ -348,6 +390,7 @@ class MriqJob(Job):
                                             self.phimag.data_ptr(), self.numk, self.numx, i["x"].data_ptr(),
                                             i["y"].data_ptr(), i["z"].data_ptr(), self.qr.data_ptr(),
                                             self.qi.data_ptr())
+        self.main_step = 1
         self.steps = [Step("mriq_phimag", (_cdiv(self.numk, 256), 1, 1), self.args_pm, 1),
                       Step("mriq_q", (_cdiv(self.numx, 256), 1, 1), self.args_q, 1)]
 
@@ -361,7 +404,7 @@ class MriqJob(Job):
 
 
 JOBS = {"mop": MopJob, "stencil": StencilJob, "histo": HistoJob, "bfs": BfsJob, "cutcp": CutcpJob,
-        "tpacf": TpacfJob, "spmv": SpmvJob, "sgemm": SgemmJob, "mriq": MriqJob}
+        "tpacf": TpacfJob, "spmv": SpmvJob, "sgemm": SgemmTcJob, "sgemm_simt": SgemmJob, "mriq": MriqJob}
 
 
 def make_job(name: str, d: dict, device="cuda") -> Job:
