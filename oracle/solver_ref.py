@@ -33,6 +33,9 @@ Readings (DESIGN.md):
               accepted nothing.
   R-solver-7  Weights w (§2.2, "changing the sharing
               ratio") scale each request's share of every total; default 1.
+  R-solver-8  A request with several kernels (mri-q, sgemm split + GEMM) is
+              represented by its main step; every other step is solved against
+              the same active set with its own kernel in the request's place.
 """
 from __future__ import annotations
 
@@ -248,12 +251,9 @@ def solve(ds: Sequence[Demand], caps: Caps = Caps()) -> list[int]:
     return n
 
 
-def step_quota(main: Demand, n_main: int, step: Demand) -> int:
-    """Quota of a secondary kernel of a multi-kernel request (R-solver-8):
-    the largest CTA count of `step` that uses no more of any resource than
-    n_main CTAs of the request's main kernel, capped by the step's G, >= 1."""
-    if step.grid_vgs == 0:
-        return 0
-    m = min((n_main * main.thr) // step.thr, (n_main * main.regs) // step.regs,
-            (n_main * main.smem) // step.smem, (n_main * main.cta) // step.cta)
-    return max(1, min(m, step.grid_vgs))
+def step_quota(ds: Sequence[Demand], i: int, step: Demand, caps: Caps = Caps()) -> int:
+    """Quota of a secondary kernel of request i (R-solver-8): the same active
+    set solved again with request i represented by that step's own kernel."""
+    dj = list(ds)
+    dj[i] = step
+    return solve(dj, caps)[i]

@@ -81,7 +81,8 @@ struct alignas(128) Desc {
   uint32_t admit_fail;   // RESOLVE: CTAs refused at admission
   uint32_t evicted;      // RESOLVE: CTAs that left at a dequeue (shrink)
   uint32_t last_live;    // RESOLVE: live quota seen by the last refused CTA
-  uint32_t pad2[20];
+  uint32_t adm;          // RESOLVE: admission tickets (alive + in-flight refusals)
+  uint32_t pad2[19];
 };
 static_assert(sizeof(Desc) == 384, "Desc layout");
 
@@ -111,6 +112,12 @@ __device__ __forceinline__ unsigned long long globaltimer() {
   unsigned long long t;
   asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
   return t;
+}
+
+__device__ __forceinline__ uint32_t ld_relaxed(const uint32_t* p) {
+  uint32_t v;
+  asm volatile("ld.relaxed.gpu.global.u32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
+  return v;
 }
 
 __device__ __forceinline__ uint32_t ld_volatile(const uint32_t* p) {
@@ -189,40 +196,49 @@ enum : uint32_t {
   kCfgStride = 1u << 19
 };
 
-// Master work-item, admission into launch d under RESOLVE (count-based):
-// returns false if the launch already holds `live` CTAs.
+// Master work-item, admission into launch d under RESOLVE (count-based).
+// Two counters: `adm` hands out tickets (a refused CTA gives its ticket back,
+// so adm can be transiently high -- at worst a concurrent arrival is refused
+// spuriously), `alive` counts admitted CTAs exactly and is what eviction
+// reads (an atomicAdd/atomicSub pair on `alive` itself made admitted CTAs see a
+// transient alive > live and evict themselves; a CAS loop on it serialised
+// hundreds of CTAs at every launch start).
 __device__ __forceinline__ bool admit(Desc* d) {
-  // compare-and-swap, so a refused CTA never inflates `alive` (an atomicAdd
-  // followed by an atomicSub would make admitted CTAs see a transient
-  // alive > live and evict themselves)
-  const uint32_t live = ld_volatile(&d->ctl->live);
-  uint32_t a = ld_volatile(&d->alive);
-  for (;;) {
-    if (a >= live) {
-      red_add_u32(&d->admit_fail, 1u);
-      d->last_live = live;
-      return false;
-    }
-    const uint32_t prev = atomicCAS(&d->alive, a, a + 1u);
-    if (prev == a) break;
-    a = prev;
+  const uint32_t live = ld_relaxed(&d->ctl->live);
+  const uint32_t t = atomicAdd(&d->adm, 1u);
+  if (t >= live) {
+    red_add_u32(&d->adm, 0xffffffffu);   // -1
+    red_add_u32(&d->admit_fail, 1u);
+    d->last_live = live;
+    return false;
   }
-  atomicMax(&d->max_alive, a + 1u);
+  const uint32_t a = atomicAdd(&d->alive, 1u) + 1u;
+  asm volatile("red.relaxed.gpu.global.max.u32 [%0], %1;" ::"l"(&d->max_alive), "r"(a) : "memory");
   __threadfence();  // admission visible before the first dequeue
   return true;
 }
+
+// Per-CTA (thread 0) view of the live quota and the admitted count, loaded
+// right after each dequeue and used at the next one, so the RESOLVE check
+// adds no latency in front of the queue atomic.
+struct AdmHint {
+  uint32_t live = 0xffffffffu;
+  uint32_t alive = 0;
+};
 
 // One dequeue (Fig. 8b line 26, rt_sched_wgroup): under RESOLVE a CTA
 // leaves first if the launch holds more CTAs than the live quota (shrink at a
 // VG boundary; CAS so exactly alive - live CTAs leave); then one atomicAdd of
 // `chunk` on the queue head.
-__device__ __forceinline__ uint32_t dequeue(Desc* d, uint32_t chunk, bool resolve, bool& admitted) {
-  if (resolve) {
-    const uint32_t live = ld_volatile(&d->ctl->live);
-    uint32_t a = ld_volatile(&d->alive);
+__device__ __forceinline__ uint32_t dequeue(Desc* d, uint32_t chunk, bool resolve, bool& admitted,
+                                            AdmHint& hint) {
+  if (resolve && hint.alive > hint.live) {
+    uint32_t live = ld_relaxed(&d->ctl->live);
+    uint32_t a = ld_relaxed(&d->alive);
     while (a > live) {
       const uint32_t prev = atomicCAS(&d->alive, a, a - 1u);
       if (prev == a) {
+        red_add_u32(&d->adm, 0xffffffffu);
         red_add_u32(&d->evicted, 1u);
         admitted = false;
         return kTerminate;
@@ -230,13 +246,19 @@ __device__ __forceinline__ uint32_t dequeue(Desc* d, uint32_t chunk, bool resolv
       a = prev;
     }
   }
-  return atomicAdd(&d->next, chunk);
+  const uint32_t b = atomicAdd(&d->next, chunk);
+  if (resolve) {
+    hint.live = ld_relaxed(&d->ctl->live);
+    hint.alive = ld_relaxed(&d->alive);
+  }
+  return b;
 }
 
 __device__ __forceinline__ void retire(Desc* d, uint32_t cfg, bool admitted) {
   if ((cfg & kCfgResolve) && admitted) {
     __threadfence();  // this CTA's VG results before the alive decrement
     atomicSub(&d->alive, 1u);
+    red_add_u32(&d->adm, 0xffffffffu);
   }
   if (cfg & kCfgStamps) red_max_u64(&d->t_last, globaltimer());
 }
@@ -261,6 +283,7 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
   const bool resolve = (cfg & kCfgResolve) != 0;
   const bool stride = !resolve && (cfg & kCfgStride) != 0;
   bool admitted = true;      // meaningful in thread 0 only
+  AdmHint hint;              // thread 0, RESOLVE
   uint32_t iter = 0;         // stride ablation: chunks taken so far (thread 0)
   if (threadIdx.x == 0) {    // master work-item: environment init (rt_env_init)
     uint32_t b = kTerminate;
@@ -270,11 +293,11 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     if (cfg & kCfgStamps) red_min_u64(&d->t_first, globaltimer());
     const uint32_t launch_idx = d->launch_idx;
     const uint32_t total = vg_total<T>(args, d, launch_idx);
-    if (blockIdx.x == 0 || resolve) d->total_seen = total;
+    if (blockIdx.x == 0) d->total_seen = total;
     if (resolve) {
-      atomicMax(&d->ctl->cur, d->req_idx);
+      asm volatile("red.relaxed.gpu.global.max.u32 [%0], %1;" ::"l"(&d->ctl->cur), "r"(d->req_idx) : "memory");
       admitted = admit(d);
-      if (admitted) b = dequeue(d, chunk, true, admitted);
+      if (admitted) b = dequeue(d, chunk, true, admitted, hint);
     }
     if (b < total) red_add_u32(&d->ctas_started, 1u);
     S->cur = b;
@@ -295,7 +318,7 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     if (threadIdx.x == 0 && !have_nxt) {
       // prefetch the next chunk id once per chunk, early (hidden behind the body)
       if (stride) nxt = (blockIdx.x + (++iter) * gridDim.x) * chunk;
-      else nxt = dequeue(d, chunk, resolve, admitted);
+      else nxt = dequeue(d, chunk, resolve, admitted, hint);
       have_nxt = true;
     }
     T::body(args, decode(vg, S->gx, S->gy, S->gz, S->launch_idx), smem);

@@ -120,7 +120,7 @@ struct DescHost {
   uint32_t next, pad1[31];
   // line 2
   unsigned long long t_first, t_last;
-  uint32_t total_seen, ctas_started, alive, max_alive, topped, admit_fail, evicted, last_live, pad2[20];
+  uint32_t total_seen, ctas_started, alive, max_alive, topped, admit_fail, evicted, last_live, adm, pad2[19];
 };
 static_assert(sizeof(DescHost) == accel::kDescBytes, "host view of the descriptor");
 

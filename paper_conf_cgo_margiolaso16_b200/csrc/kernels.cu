@@ -50,6 +50,10 @@ __global__ void desc_init_kernel(const InitParams p, uint32_t n_desc) {
   d->ctas_started = 0;
   d->alive = 0;
   d->max_alive = 0;
+  d->adm = 0;
+  d->admit_fail = 0;
+  d->evicted = 0;
+  d->last_live = 0;
   d->topped = 0;
   d->req_idx = i;
   d->has_prev = i > 0 ? 1u : 0u;

@@ -168,9 +168,10 @@ def test_zero_grid_gets_zero():
 
 
 def test_step_quota():
+    """R-solver-8: a secondary step is solved with its own kernel in place."""
     main = S.demand_of(256, 32, 0, 10 ** 6)
+    other = S.demand_of(256, 32, 0, 10 ** 6)
     small = S.demand_of(256, 32, 0, 8)
-    assert S.step_quota(main, 296, small) == 8
-    other = S.demand_of(128, 32, 0, 10 ** 6)
-    # half the threads/regs, but the same 1 KiB reserved smem and 1 CTA slot each
-    assert S.step_quota(main, 296, other) == 296
+    assert S.step_quota([main, other], 0, small) == 8
+    big_smem = S.demand_of(128, 96, 190 * 1024, 256)
+    assert S.step_quota([main, other], 0, big_smem) == 148  # one 191-KB CTA per SM
