@@ -95,7 +95,8 @@ const char *accel_last_error(const accel_ctx *ctx);
  * its block shape.  The block shape is never changed. */
 typedef struct {
   const char *name;
-  const void *persistent_fn;  /* host stub of accel_persistent<T>              */
+  const void *persistent_fn;  /* host stub of accel_persistent<T, STATIC>      */
+  const void *persistent_resolve_fn; /* accel_persistent<T, RESOLVE>; NULL = persistent_fn */
   const void *native_fn;      /* host stub of accel_native<T>                  */
   const void *topup_fn;       /* host stub of accel_topup<T> (RESOLVE growth)  */
   accel_dim3 block;           /* work-group (CTA) shape                        */

@@ -32,9 +32,8 @@ typedef struct {
  * grid (ceil(nx/128), ceil(ny/8), ceil(nz/8)).  Launch r reads
  * (r == 0 ? a0 : buf[(r-1)&1]) and writes buf[r&1]; after T launches the
  * result is in buf[(T-1)&1].  Interior: c1*(6-neighbour sum) - c0*a;
- * faces copy the input.  Layout contract: each of a0/buf0/buf1 points at plane
- * 0 of an allocation with one extra plane (nx*ny floats) before it and three
- * after plane nz-1 (halo and prefetch loads stay in bounds; values unused). */
+ * faces copy the input.  a0/buf0/buf1: DEVICE pointers to nx*ny*nz floats,
+ * 16-B aligned, no padding required. */
 typedef struct {
   const float *a0;
   float *buf0;

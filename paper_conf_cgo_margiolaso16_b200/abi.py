@@ -46,7 +46,8 @@ class accel_config(C.Structure):
 
 
 class accel_kernel_desc(C.Structure):
-    _fields_ = [("name", C.c_char_p), ("persistent_fn", vp), ("native_fn", vp), ("topup_fn", vp),
+    _fields_ = [("name", C.c_char_p), ("persistent_fn", vp), ("persistent_resolve_fn", vp), ("native_fn", vp),
+                ("topup_fn", vp),
                 ("block", accel_dim3),
                 ("dyn_smem", u32), ("regs", i32), ("chunk", u32), ("args_size", u32)]
 

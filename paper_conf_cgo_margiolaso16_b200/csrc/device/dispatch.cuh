@@ -82,7 +82,8 @@ struct alignas(128) Desc {
   uint32_t evicted;      // RESOLVE: CTAs that left at a dequeue (shrink)
   uint32_t last_live;    // RESOLVE: live quota seen by the last refused CTA
   uint32_t adm;          // RESOLVE: admission tickets (alive + in-flight refusals)
-  uint32_t pad2[19];
+  uint32_t draining;     // RESOLVE: evicted CTAs still finishing their last VG
+  uint32_t pad2[18];
 };
 static_assert(sizeof(Desc) == 384, "Desc layout");
 
@@ -178,22 +179,27 @@ __device__ __forceinline__ void wait_complete(const Desc* p) {
     const uint32_t tot = ld_volatile(&p->total_seen);
     if (tot != kTerminate && ld_volatile(&p->next) >= tot) {
       __threadfence();
-      if (ld_volatile(&p->alive) == 0) break;
+      if (ld_volatile(&p->alive) == 0) {
+        __threadfence();
+        if (ld_volatile(&p->draining) == 0) break;
+      }
     }
     __nanosleep(256);
   }
   __threadfence();
+  // the launch's results were written through the generic proxy by other CTAs;
+  // this CTA may read them with TMA (async proxy)
+  asm volatile("fence.proxy.async.global;" ::: "memory");
 }
 
 // Launch configuration word, a kernel parameter (no descriptor load on the
-// critical path of a CTA's first dequeue): bits 0-15 chunk, then flags.
-//   kCfgStride: static round-robin VG assignment (VG = cta + i * grid), no
-//               queue -- an ablation to measure the cost of the dynamic queue.
+// critical path of a CTA's first dequeue): bits 0-15 chunk, then flags.  The
+// policy itself is a template parameter, so the STATIC kernel carries no
+// RESOLVE state in its registers.
 enum : uint32_t {
   kCfgChunkMask = 0xffffu,
   kCfgResolve = 1u << 16,
-  kCfgStamps = 1u << 17,
-  kCfgStride = 1u << 19
+  kCfgStamps = 1u << 17
 };
 
 // Master work-item, admission into launch d under RESOLVE (count-based).
@@ -229,36 +235,50 @@ struct AdmHint {
 // One dequeue (Fig. 8b line 26, rt_sched_wgroup): under RESOLVE a CTA
 // leaves first if the launch holds more CTAs than the live quota (shrink at a
 // VG boundary; CAS so exactly alive - live CTAs leave); then one atomicAdd of
-// `chunk` on the queue head.
-__device__ __forceinline__ uint32_t dequeue(Desc* d, uint32_t chunk, bool resolve, bool& admitted,
+// `chunk` on the queue head.  The dequeue is a prefetch issued while the CTA's
+// current VG is still running, so an evicted CTA is `draining` (counted by
+// wait_complete) until retire(), after that VG's results are written.
+template <bool kResolve>
+__device__ __forceinline__ uint32_t dequeue(Desc* d, uint32_t chunk, bool& admitted, bool& draining,
                                             AdmHint& hint) {
-  if (resolve && hint.alive > hint.live) {
+  if (kResolve && hint.alive > hint.live) {
     uint32_t live = ld_relaxed(&d->ctl->live);
     uint32_t a = ld_relaxed(&d->alive);
-    while (a > live) {
-      const uint32_t prev = atomicCAS(&d->alive, a, a - 1u);
-      if (prev == a) {
-        red_add_u32(&d->adm, 0xffffffffu);
-        red_add_u32(&d->evicted, 1u);
-        admitted = false;
-        return kTerminate;
+    if (a > live) {
+      atomicAdd(&d->draining, 1u);
+      __threadfence();   // draining visible before alive drops
+      while (a > live) {
+        const uint32_t prev = atomicCAS(&d->alive, a, a - 1u);
+        if (prev == a) {
+          red_add_u32(&d->adm, 0xffffffffu);
+          red_add_u32(&d->evicted, 1u);
+          admitted = false;
+          draining = true;
+          return kTerminate;
+        }
+        a = prev;
       }
-      a = prev;
+      red_add_u32(&d->draining, 0xffffffffu);   // not evicted after all
     }
   }
   const uint32_t b = atomicAdd(&d->next, chunk);
-  if (resolve) {
+  if (kResolve) {
     hint.live = ld_relaxed(&d->ctl->live);
     hint.alive = ld_relaxed(&d->alive);
   }
   return b;
 }
 
-__device__ __forceinline__ void retire(Desc* d, uint32_t cfg, bool admitted) {
-  if ((cfg & kCfgResolve) && admitted) {
+template <bool kResolve>
+__device__ __forceinline__ void retire(Desc* d, uint32_t cfg, bool admitted, bool draining) {
+  if (kResolve && admitted) {
     __threadfence();  // this CTA's VG results before the alive decrement
     atomicSub(&d->alive, 1u);
     red_add_u32(&d->adm, 0xffffffffu);
+  }
+  if (kResolve && draining) {
+    __threadfence();  // the last VG's results before the draining decrement
+    atomicSub(&d->draining, 1u);
   }
   if (cfg & kCfgStamps) red_max_u64(&d->t_last, globaltimer());
 }
@@ -267,40 +287,49 @@ __device__ __forceinline__ void retire(Desc* d, uint32_t cfg, bool admitted) {
 // Fig. 8b).  Keeping it in shared memory instead of registers
 // leaves the body the same register budget it has in the native kernel: only
 // the current VG id and the prefetched chunk id live across the body call.
+// The VG to run next is double-buffered: thread 0 publishes VG k+1 into
+// cur[(k+1)&1] while slower warps may still be loading cur[k&1] (a body
+// need not contain a barrier); the barrier closing iteration k orders both.
 struct SchedState {
-  uint32_t cur;        // VG to run next (sd.wg_base)
+  struct Cur {
+    uint32_t vg;         // VG to run next (sd.wg_base)
+    uint32_t x, y, z;    // its decode, by thread 0 (the warps only load it)
+  } cur[2];
   uint32_t end;        // end of the current chunk (sd.wg_end)
-  uint32_t total;      // VGs of this launch (RUN_TERMINATE when cur >= total)
+  uint32_t total;      // VGs of this launch (RUN_TERMINATE when vg >= total)
   uint32_t gx, gy, gz, launch_idx;
   uint32_t* coverage;
+  __device__ __forceinline__ void set_cur(uint32_t k, uint32_t vg) {
+    cur[k].vg = vg;
+    if (vg < total) {
+      const VirtualBlock b = decode(vg, gx, gy, gz, launch_idx);
+      cur[k].x = b.x; cur[k].y = b.y; cur[k].z = b.z;
+    }
+  }
 };
 
 // Serve one launch: admission, dequeue loop, retire.  All threads call it.
-template <class T>
+template <class T, bool kResolve>
 __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, char* smem,
                                       SchedState* S, uint32_t cfg) {
   const uint32_t chunk = cfg & kCfgChunkMask;
-  const bool resolve = (cfg & kCfgResolve) != 0;
-  const bool stride = !resolve && (cfg & kCfgStride) != 0;
   bool admitted = true;      // meaningful in thread 0 only
-  AdmHint hint;              // thread 0, RESOLVE
-  uint32_t iter = 0;         // stride ablation: chunks taken so far (thread 0)
+  bool draining = false;     // thread 0: evicted at the prefetch, last VG in flight
+  AdmHint hint;              // thread 0, RESOLVE only
   if (threadIdx.x == 0) {    // master work-item: environment init (rt_env_init)
     uint32_t b = kTerminate;
     // STATIC: the first dequeue is issued before anything else is loaded
-    if (stride) b = blockIdx.x * chunk;
-    else if (!resolve) b = atomicAdd(&d->next, chunk);
+    if (!kResolve) b = atomicAdd(&d->next, chunk);
     if (cfg & kCfgStamps) red_min_u64(&d->t_first, globaltimer());
     const uint32_t launch_idx = d->launch_idx;
     const uint32_t total = vg_total<T>(args, d, launch_idx);
     if (blockIdx.x == 0) d->total_seen = total;
-    if (resolve) {
+    if (kResolve) {
       asm volatile("red.relaxed.gpu.global.max.u32 [%0], %1;" ::"l"(&d->ctl->cur), "r"(d->req_idx) : "memory");
       admitted = admit(d);
-      if (admitted) b = dequeue(d, chunk, true, admitted, hint);
+      if (admitted) b = dequeue<true>(d, chunk, admitted, draining, hint);
     }
     if (b < total) red_add_u32(&d->ctas_started, 1u);
-    S->cur = b;
     S->end = b < total ? min(b + chunk, total) : b;
     S->total = total;
     S->gx = d->gx;
@@ -308,48 +337,54 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     S->gz = d->gz;
     S->launch_idx = launch_idx;
     S->coverage = d->coverage;
+    S->set_cur(0, b);
   }
   __syncthreads();
   uint32_t nxt = kTerminate;  // thread 0: id of the next chunk, requested at chunk start
   bool have_nxt = false;
-  for (;;) {
-    const uint32_t vg = S->cur;
+  for (uint32_t k = 0;; k ^= 1u) {
+    const SchedState::Cur c = S->cur[k];
+    const uint32_t vg = c.vg;
     if (vg >= S->total) break;                 // RUN_TERMINATE
     if (threadIdx.x == 0 && !have_nxt) {
       // prefetch the next chunk id once per chunk, early (hidden behind the body)
-      if (stride) nxt = (blockIdx.x + (++iter) * gridDim.x) * chunk;
-      else nxt = dequeue(d, chunk, resolve, admitted, hint);
+      nxt = dequeue<kResolve>(d, chunk, admitted, draining, hint);
       have_nxt = true;
     }
-    T::body(args, decode(vg, S->gx, S->gy, S->gz, S->launch_idx), smem);
+    VirtualBlock vb;
+    vb.x = c.x; vb.y = c.y; vb.z = c.z;
+    vb.gx = S->gx; vb.gy = S->gy; vb.gz = S->gz;
+    vb.linear = vg;
+    vb.launch_idx = S->launch_idx;
+    T::body(args, vb, smem);
     if (threadIdx.x == 0) {
       if (S->coverage != nullptr) atomicAdd(&S->coverage[vg], 1u);
       if (vg + 1 < S->end) {
-        S->cur = vg + 1;
+        S->set_cur(k ^ 1u, vg + 1);
       } else {                                   // publish the prefetched chunk
-        S->cur = nxt;
         S->end = nxt < S->total ? min(nxt + chunk, S->total) : nxt;
+        S->set_cur(k ^ 1u, nxt);
         have_nxt = false;
       }
     }
     __syncthreads();
   }
-  if (threadIdx.x == 0) retire(d, cfg, admitted);
+  if (threadIdx.x == 0) retire<kResolve>(d, cfg, admitted, draining);
 }
 
 // -------------------------------------------------------------------------
 // The scheduling kernel: grid = quota (1-D), block = the original block;
-// serves launch d.  cfg = chunk | kCfg* flags.
-template <class T>
+// serves launch d.  cfg = chunk | kCfg* flags.  kResolve = RESOLVE policy.
+template <class T, bool kResolve>
 __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
     accel_persistent(const typename T::Args args, Desc* __restrict__ d, uint32_t cfg) {
   extern __shared__ __align__(128) char smem[];
   __shared__ SchedState S;
-  if (cfg & kCfgResolve) {
+  if (kResolve) {
     if (threadIdx.x == 0 && d->has_prev && ld_volatile(&(d - 1)->topped)) wait_complete(d - 1);
     __syncthreads();
   }
-  serve<T>(args, d, smem, &S, cfg);
+  serve<T, kResolve>(args, d, smem, &S, cfg);
 }
 
 // RESOLVE top-up grid: d = first launch of the request step, `sticky` =
@@ -375,7 +410,7 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
     }
     __syncthreads();
     const uint32_t cfg = dl->chunk | kCfgResolve | ((dl->flags & kFlagStamps) ? kCfgStamps : 0u);
-    serve<T>(args, dl, smem, &S, cfg);
+    serve<T, true>(args, dl, smem, &S, cfg);
     __syncthreads();
   }
 }

@@ -38,7 +38,8 @@ constexpr uint32_t kFlagStamps = 1u, kFlagAlive = 2u;  // dispatch.cuh
 
 struct Kernel {
   std::string name;
-  const void* pfn;
+  const void* pfn;   // accel_persistent<T, STATIC>
+  const void* prfn;  // accel_persistent<T, RESOLVE>
   const void* nfn;
   const void* tfn;
   dim3 block;
@@ -120,7 +121,7 @@ struct DescHost {
   uint32_t next, pad1[31];
   // line 2
   unsigned long long t_first, t_last;
-  uint32_t total_seen, ctas_started, alive, max_alive, topped, admit_fail, evicted, last_live, adm, pad2[19];
+  uint32_t total_seen, ctas_started, alive, max_alive, topped, admit_fail, evicted, last_live, adm, draining, pad2[18];
 };
 static_assert(sizeof(DescHost) == accel::kDescBytes, "host view of the descriptor");
 
@@ -303,7 +304,7 @@ int enqueue(accel_ctx* ctx, Request* r) {
       uint32_t cfg = (k.chunk & 0xffffu) | (resolve ? (1u << 16) : 0u) | (1u << 17) | ctx->dispatch_bits;
       void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &cfg};
       const dim3 grid = shared ? dim3(st.quota, 1, 1) : dim3(st.grid.x, st.grid.y, st.grid.z);
-      CK(ctx, cudaLaunchKernel(shared ? k.pfn : k.nfn, grid, k.block, params, k.dyn_smem, s));
+      CK(ctx, cudaLaunchKernel(shared ? (resolve ? k.prfn : k.pfn) : k.nfn, grid, k.block, params, k.dyn_smem, s));
     }
   }
   if (lev) CK(ctx, cudaEventRecord(r->ev_launch[li], s));
@@ -629,6 +630,7 @@ int accel_kernel_register(accel_ctx* ctx, const accel_kernel_desc* d, int32_t* k
   Kernel k;
   k.name = d->name ? d->name : "?";
   k.pfn = d->persistent_fn;
+  k.prfn = d->persistent_resolve_fn ? d->persistent_resolve_fn : d->persistent_fn;
   k.nfn = d->native_fn;
   k.tfn = d->topup_fn ? d->topup_fn : d->persistent_fn;
   k.block = dim3(d->block.x, d->block.y ? d->block.y : 1, d->block.z ? d->block.z : 1);
@@ -638,9 +640,13 @@ int accel_kernel_register(accel_ctx* ctx, const accel_kernel_desc* d, int32_t* k
   cudaFuncAttributes a;
   CK(ctx, cudaFuncGetAttributes(&a, k.pfn));
   if ((int)k.threads() > a.maxThreadsPerBlock) return ctx->fail(ACCEL_ENOFIT, "block larger than the kernel allows");
-  k.num_regs = d->regs > 0 ? d->regs : a.numRegs;
-  k.static_smem = (int)a.sharedSizeBytes;
-  for (const void* fn : {k.pfn, k.nfn, k.tfn}) {
+  cudaFuncAttributes ar;
+  CK(ctx, cudaFuncGetAttributes(&ar, k.prfn));
+  // the solver uses the larger of the two persistent instances (the one a
+  // request runs depends on the policy at submit time)
+  k.num_regs = d->regs > 0 ? d->regs : std::max(a.numRegs, ar.numRegs);
+  k.static_smem = (int)std::max(a.sharedSizeBytes, ar.sharedSizeBytes);
+  for (const void* fn : {k.pfn, k.prfn, k.nfn, k.tfn}) {
     if (k.dyn_smem > 48 * 1024)
       CK(ctx, cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)k.dyn_smem));
     // one carveout for every tenant so CTAs of different kernels can share an SM

@@ -53,6 +53,7 @@ __global__ void desc_init_kernel(const InitParams p, uint32_t n_desc) {
   d->adm = 0;
   d->admit_fail = 0;
   d->evicted = 0;
+  d->draining = 0;
   d->last_live = 0;
   d->topped = 0;
   d->req_idx = i;
@@ -80,7 +81,8 @@ template <class T>
 accel_kernel_desc make_desc(const char* name) {
   accel_kernel_desc d;
   d.name = name;
-  d.persistent_fn = reinterpret_cast<const void*>(&accel_persistent<T>);
+  d.persistent_fn = reinterpret_cast<const void*>(&accel_persistent<T, false>);
+  d.persistent_resolve_fn = reinterpret_cast<const void*>(&accel_persistent<T, true>);
   d.native_fn = reinterpret_cast<const void*>(&accel_native<T>);
   d.topup_fn = reinterpret_cast<const void*>(&accel_topup<T>);
   d.block = accel_dim3{(uint32_t)T::kThreads, 1u, 1u};

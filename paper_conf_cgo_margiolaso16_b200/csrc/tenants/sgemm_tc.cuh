@@ -26,42 +26,14 @@
 
 #include "../device/dispatch.cuh"
 #include "accel_tenants.h"
+#include "tma.cuh"
 
 namespace accel {
 
 namespace tc {
 
-__device__ __forceinline__ uint32_t smem_u32(const void* p) {
-  return static_cast<uint32_t>(__cvta_generic_to_shared(p));
-}
-__device__ __forceinline__ void mbar_init(uint32_t bar, uint32_t count) {
-  asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(bar), "r"(count) : "memory");
-}
-__device__ __forceinline__ void mbar_expect_tx(uint32_t bar, uint32_t bytes) {
-  asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(bar), "r"(bytes) : "memory");
-}
-// Wait for the phase with parity `parity` to complete; a watchdog turns a
-// protocol bug into a trap (ACCEL_ESTATE) instead of a hung GPU.
-__device__ __forceinline__ void mbar_wait(uint32_t bar, uint32_t parity) {
-  uint32_t done = 0;
-  for (uint64_t spin = 0;; ++spin) {
-    asm volatile(
-        "{\n\t.reg .pred p;\n\t"
-        "mbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2;\n\t"
-        "selp.u32 %0, 1, 0, p;\n\t}"
-        : "=r"(done)
-        : "r"(bar), "r"(parity)
-        : "memory");
-    if (done) return;
-    if (spin > (1ull << 26)) __trap();
-  }
-}
-__device__ __forceinline__ void tma_load_2d(uint32_t dst, const void* tmap, int32_t c0, int32_t c1, uint32_t bar) {
-  asm volatile(
-      "cp.async.bulk.tensor.2d.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1, {%2, %3}], [%4];" ::"r"(dst),
-      "l"(tmap), "r"(c0), "r"(c1), "r"(bar)
-      : "memory");
-}
+using namespace accel::tma;
+
 // UMMA shared-memory matrix descriptor, K-major, 128-B swizzle: rows of 128 B,
 // 8-row groups 1024 B apart (SBO), LBO = 16 B (unused for SW128 K-major),
 // version 1 (sm_100), layout type 2 = SWIZZLE_128B.
@@ -81,9 +53,6 @@ __device__ __forceinline__ void mma_tf32(uint32_t d_tmem, uint64_t adesc, uint64
 __device__ __forceinline__ void mma_commit(uint32_t bar) {
   asm volatile("tcgen05.commit.cta_group::1.mbarrier::arrive::one.shared::cluster.b64 [%0];" ::"r"(bar)
                : "memory");
-}
-__device__ __forceinline__ void mbar_arrive(uint32_t bar) {
-  asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(bar) : "memory");
 }
 __device__ __forceinline__ void fence_before() { asm volatile("tcgen05.fence::before_thread_sync;" ::: "memory"); }
 __device__ __forceinline__ void fence_after() { asm volatile("tcgen05.fence::after_thread_sync;" ::: "memory"); }
@@ -197,6 +166,8 @@ struct SgemmTc {
 
     if (warp == 0 && lane == 0) {
       // ---- TMA producer
+#pragma unroll
+      for (int q = 0; q < 4; ++q) tmap_acquire(&maps[q]);
       for (int kb = 0; kb < nk; ++kb) {
         const int s = kb % kStages;
         if (kb >= kStages) mbar_wait(empty(s), ((kb / kStages) - 1) & 1);

@@ -3,21 +3,26 @@
 //
 // One VG = a 128 x 8 x 8 (x, y, z) tile; 256 threads = 8 warps, warp w owns
 // row y0+w, lane l owns x0+4l..x0+4l+3 (one 16-B vector).  The tile is walked
-// along z (fully unrolled, so the register rotation of the column
-// z-1, z, z+1 costs nothing) with loads issued three planes ahead (HBM latency
-// ~1 us needs ~40 KB in flight per SM).  y neighbours come from a
-// double-buffered shared-memory plane of 10 rows (8 own rows + 2 halo rows),
-// x neighbours from warp shuffles plus one scalar edge load per row end.  One
-// __syncthreads per plane.
+// along z (fully unrolled: ring slots and group counts are compile-time).
+// Plane tiles (10 rows y0-1..y0+8 x 136 columns x0-4..x0+131: the tile plus
+// its y and x halos) are staged in shared memory by cp.async (16-B LDGSTS,
+// L2-only), kD planes ahead into a ring of kR slots, one commit group per
+// plane and ONE __syncthreads per plane.  Out-of-volume pieces are
+// zero-filled (src-size 0); they only feed face cells, which copy the input.
+// The column z-1, z, z+1 of each thread lives in registers; y neighbours and
+// the two x edges come from the staged plane, inner x neighbours from warp
+// shuffles.  Occupancy is set by shared memory (6 CTAs/SM, ~130 KB in flight
+// per SM).  Algorithmic traffic: 8 B per point per sweep.
 //
-// Layout contract (include/accel_tenants.h): every volume has one readable
-// plane before z = 0 and three after z = nz-1, so the halo / prefetch loads
-// at the domain faces are plain in-bounds loads (their values only feed face
-// cells, which copy the input) and the loop body has no bounds logic at all.
-// Algorithmic traffic: 8 B per point per sweep.
+// A TMA (cp.async.bulk.tensor.2d) staging of the same tiles was 14 % faster
+// in isolation but returned stale tile data when it ran concurrently with
+// the bfs tenant (boxes partially outside the volume at the x faces; never
+// reproduced in isolation or for the sgemm tenant's in-bounds boxes) -- see
+// DESIGN.md, "stencil staging".
 #pragma once
 #include "../device/dispatch.cuh"
 #include "accel_tenants.h"
+#include "tma.cuh"
 
 namespace accel {
 
@@ -26,90 +31,127 @@ struct Stencil {
   static constexpr int kThreads = 256;
   static constexpr int kTX = 128, kTY = 8, kTZ = 8;
   static constexpr uint32_t kChunk = 1;
-  static constexpr int kMinBlocks = 4;     // <= 64 regs: 32 warps/SM in both modes
-  static constexpr int kRows = kTY + 2;
-  static constexpr uint32_t kDynSmem = 2 * kRows * kTX * sizeof(float);  // 10 KB
+  static constexpr int kMinBlocks = 6;
+  static constexpr int kRows = kTY + 2;                 // y halo
+  static constexpr int kCols = kTX + 8;                 // x0-4 .. x0+131 (16-B multiples)
+  static constexpr uint32_t kPlaneBytes = kRows * kCols * 4;          // 5440
+  static constexpr uint32_t kSlot = (kPlaneBytes + 127) / 128 * 128;  // 5504
+#ifndef STENCIL_KD
+#define STENCIL_KD 3
+#endif
+  static constexpr int kD = STENCIL_KD;                 // planes in flight beyond z+1
+  static constexpr int kR = kD + 2;                     // ring slots
+  static constexpr uint32_t kDynSmem = kR * kSlot + 128;   // + alignment
 
-  static __device__ __forceinline__ float4 ld4(const float* p) {
-    return __ldg(reinterpret_cast<const float4*>(p));
-  }
-
-  static __device__ __forceinline__ void body(const Args& a, const VirtualBlock& vb, char* smem) {
+  // cp.async (LDGSTS, 16 B per copy, L2-only .cg) staging: every thread
+  // copies <= 2 of the 340 16-B pieces of a plane tile; out-of-volume pieces are
+  // zero-filled (src-size 0).  One commit group per plane, planes kD ahead.
+  static __device__ __forceinline__ void body(const Args& a, const VirtualBlock& vb, char* smem_raw) {
+    using namespace tma;
     const uint32_t r = vb.launch_idx;
     const float* __restrict__ in = r == 0 ? a.a0 : ((r & 1) ? a.buf0 : a.buf1);
     float* __restrict__ out = (r & 1) ? a.buf1 : a.buf0;
     const int nx = (int)a.nx, ny = (int)a.ny, nz = (int)a.nz;
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
-    const int x0 = (int)vb.x * kTX + 4 * lane;
+    const int x0 = (int)vb.x * kTX;
     const int y0 = (int)vb.y * kTY;
     const int y = y0 + warp;
     const int z0 = (int)vb.z * kTZ;
-    const int nzt = min(kTZ, nz - z0);     // planes in this tile (ragged last tile)
-    const int plane = nx * ny;
-    const bool active = x0 < nx && y < ny;
-    // rows beyond the domain in x or y read an in-range neighbour row (clamped
-    // once); z never needs clamping thanks to the padding planes
-    const int xc = min(x0, nx - 4);
-    const int col = min(y, ny - 1) * nx + xc;
-    const bool hown = warp == 0 || warp == kTY - 1;
-    const int hrow = warp == 0 ? 0 : kRows - 1;
-    const int hcol = min(warp == 0 ? y0 - 1 : y0 + kTY, ny - 1) * nx + xc;  // y0-1 = -1 is padding
-    const bool eown = lane == 0 || lane == 31;
-    const int ecol = min(y, ny - 1) * nx + (lane == 0 ? x0 - 1 : min(x0 + 4, nx - 1));
-    const float* pc = in + z0 * plane + col;   // own column at plane z0
-    const float* ph = in + z0 * plane + hcol;
-    const float* pe = in + z0 * plane + ecol;
-    float* po = out + z0 * plane + y * nx + x0;
+    const int nzt = min(kTZ, nz - z0);
+    const int nplanes = nzt + 2;
+    const uint32_t sbase = (smem_u32(smem_raw) + 127u) & ~127u;
+    const int rows_total = nz * ny;
+    const int row0 = (z0 - 1) * ny + y0 - 1;            // matrix row of plane 0's first row
+    // my two pieces: e = tid, tid + 256 (< 340); piece e = row e / 34, 16-B column e % 34
+    constexpr int kPieces = kRows * (kCols / 4);
+    const int e0 = threadIdx.x, e1 = threadIdx.x + kThreads;
+    const bool has1 = e1 < kPieces;
+    const int rr0 = e0 / (kCols / 4), c0x = x0 - 4 + 4 * (e0 % (kCols / 4));
+    const int rr1 = e1 / (kCols / 4), c1x = x0 - 4 + 4 * (e1 % (kCols / 4));
+    const bool colok0 = c0x >= 0 && c0x < nx, colok1 = has1 && c1x >= 0 && c1x < nx;
+    const uint32_t soff0 = 16u * (uint32_t)e0, soff1 = 16u * (uint32_t)e1;
+    auto issue = [&](int p) {
+      const uint32_t dst = sbase + (uint32_t)(p % kR) * kSlot;
+      const int R0 = row0 + p * ny + rr0;
+      const bool ok0 = colok0 && R0 >= 0 && R0 < rows_total;
+      const float* s0 = ok0 ? in + (size_t)R0 * nx + c0x : in;
+      asm volatile("cp.async.cg.shared.global [%0], [%1], 16, %2;" ::"r"(dst + soff0), "l"(s0), "r"(ok0 ? 16 : 0)
+                   : "memory");
+      if (has1) {
+        const int R1 = row0 + p * ny + rr1;
+        const bool ok1 = colok1 && R1 >= 0 && R1 < rows_total;
+        const float* s1 = ok1 ? in + (size_t)R1 * nx + c1x : in;
+        asm volatile("cp.async.cg.shared.global [%0], [%1], 16, %2;" ::"r"(dst + soff1), "l"(s1), "r"(ok1 ? 16 : 0)
+                     : "memory");
+      }
+    };
+    auto commit = [] { asm volatile("cp.async.commit_group;" ::: "memory"); };
+    // prologue: planes 0 .. kD+1 (one group each, empty groups past the tile)
+#pragma unroll
+    for (int p = 0; p < kD + 2; ++p) {
+      if (p < nplanes) issue(p);
+      commit();
+    }
+    auto slot = [&](int p) { return sbase + (uint32_t)(p % kR) * kSlot; };
 
+    const bool active = x0 + 4 * lane < nx && y < ny;
     const bool yint = y >= 1 && y <= ny - 2;
     bool mxy[4];
 #pragma unroll
-    for (int e = 0; e < 4; ++e) mxy[e] = yint && (x0 + e >= 1) && (x0 + e <= nx - 2);
+    for (int e = 0; e < 4; ++e) {
+      const int x = x0 + 4 * lane + e;
+      mxy[e] = yint && x >= 1 && x <= nx - 2;
+    }
     const float c0 = a.c0, c1 = a.c1;
-
-    float4 zm = ld4(pc - plane), cur = ld4(pc), n1 = ld4(pc + plane), n2 = ld4(pc + 2 * plane);
-    float4 hc = hown ? ld4(ph) : cur;
-    float ec = eown ? __ldg(pe) : 0.f;
-    float4* S = reinterpret_cast<float4*>(smem);  // [2][kRows][32]
+    const uint32_t own = 4u * (uint32_t)((warp + 1) * kCols + 4 + 4 * lane);
+    const uint32_t edge = 4u * (uint32_t)((warp + 1) * kCols + (lane == 31 ? 4 + kTX : 3));
+    // planes 0 and 1 landed (groups 0, 1 of kD + 2 committed)
+    asm volatile("cp.async.wait_group %0;" ::"n"(kD) : "memory");
+    __syncthreads();
+    float4 zm = lds_f4(slot(0) + own);
+    float4 cur = lds_f4(slot(1) + own);
+    float* po = out + ((size_t)z0 * ny + y) * nx + x0 + 4 * lane;
+    const size_t pstride = (size_t)nx * ny;
 #pragma unroll
     for (int i = 0; i < kTZ; ++i) {
       if (i >= nzt) break;
-      const int z = z0 + i;
-      const float4 n3 = ld4(pc + (i + 3) * plane);
-      const float4 hn = hown ? ld4(ph + (i + 1) * plane) : cur;
-      const float en = eown ? __ldg(pe + (i + 1) * plane) : 0.f;
-
-      float4* Sb = S + (i & 1) * (kRows * 32);
-      Sb[(warp + 1) * 32 + lane] = cur;
-      if (hown) Sb[hrow * 32 + lane] = hc;
+      const int pz = i + 1;   // plane pz (= z) is `cur`; plane pz+1 must have landed
+      // groups committed: kD + 2 + i; plane pz+1 is group i+2, so at most
+      // kD - 1 may still be pending
+      asm volatile("cp.async.wait_group %0;" ::"n"(kD - 1) : "memory");
+      __syncthreads();        // plane pz+1 visible; every thread done with iteration i-1
+      // refill the slot of plane pz-1 (last read in iteration i-1) with plane pz+kD+1
+      if (pz + kD + 1 < nplanes) issue(pz + kD + 1);
+      commit();
+      const uint32_t P = slot(pz);
+      const float4 zp = lds_f4(slot(pz + 1) + own);
+      const float4 ym = lds_f4(P + own - 4u * kCols);
+      const float4 yp = lds_f4(P + own + 4u * kCols);
+      const float ev = lds_f32(P + edge);
       float xl = __shfl_up_sync(0xffffffffu, cur.w, 1);
       float xr = __shfl_down_sync(0xffffffffu, cur.x, 1);
-      if (lane == 0) xl = ec;
-      if (lane == 31) xr = ec;
-      __syncthreads();
-      const float4 ym = Sb[warp * 32 + lane];
-      const float4 yp = Sb[(warp + 2) * 32 + lane];
-
-      // compute every element unconditionally, then select (no branches)
-      const float vx = ((((((zm.x + n1.x) + ym.x) + yp.x) + xl) + cur.y) * c1 - cur.x * c0);
-      const float vy = ((((((zm.y + n1.y) + ym.y) + yp.y) + cur.x) + cur.z) * c1 - cur.y * c0);
-      const float vz = ((((((zm.z + n1.z) + ym.z) + yp.z) + cur.y) + cur.w) * c1 - cur.z * c0);
-      const float vw = ((((((zm.w + n1.w) + ym.w) + yp.w) + cur.z) + xr) * c1 - cur.w * c0);
+      if (lane == 0) xl = ev;
+      if (lane == 31) xr = ev;
+      const int z = z0 + i;
+      const float vx = ((((((zm.x + zp.x) + ym.x) + yp.x) + xl) + cur.y) * c1 - cur.x * c0);
+      const float vy = ((((((zm.y + zp.y) + ym.y) + yp.y) + cur.x) + cur.z) * c1 - cur.y * c0);
+      const float vz = ((((((zm.z + zp.z) + ym.z) + yp.z) + cur.y) + cur.w) * c1 - cur.z * c0);
+      const float vw = ((((((zm.w + zp.w) + ym.w) + yp.w) + cur.z) + xr) * c1 - cur.w * c0);
       const bool zint = z >= 1 && z <= nz - 2;
       float4 o;
       o.x = (zint && mxy[0]) ? vx : cur.x;
       o.y = (zint && mxy[1]) ? vy : cur.y;
       o.z = (zint && mxy[2]) ? vz : cur.z;
       o.w = (zint && mxy[3]) ? vw : cur.w;
-      if (active) *reinterpret_cast<float4*>(po + i * plane) = o;
+      if (active) *reinterpret_cast<float4*>(po) = o;
+      po += pstride;
       zm = cur;
-      cur = n1;
-      n1 = n2;
-      n2 = n3;
-      hc = hn;
-      ec = en;
+      cur = zp;
     }
+    asm volatile("cp.async.wait_all;" ::: "memory");
+    __syncthreads();   // the CTA's next VG reuses the ring
   }
+
 };
 
 }  // namespace accel

@@ -157,17 +157,11 @@ class StencilJob(Job):
         if self.nx % 4:
             raise ValueError("stencil needs nx % 4 == 0 (16-B rows)")
         n = self.nx * self.ny * self.nz
-        plane = self.nx * self.ny
-        # layout contract: 1 readable plane before z = 0, 3 after z = nz - 1
-        pad = [torch.zeros(n + 4 * plane, dtype=torch.float32, device=self.device) for _ in range(3)]
-        self._pad = pad
-        pad[0][plane:plane + n].copy_(torch.from_numpy(np.ascontiguousarray(d["a0"]).ravel()))
-        self.inputs = {"a0": pad[0][plane:plane + n]}
-        self.buf = [pad[1][plane:plane + n], pad[2][plane:plane + n]]
+        self.inputs = {"a0": _dev(d["a0"].ravel(), self.device)}
+        self.buf = [torch.empty(n, dtype=torch.float32, device=self.device) for _ in range(2)]
         self.out = {"a": self.buf[(self.sweeps - 1) & 1]}
         self.args = abi.accel_stencil_args(self.inputs["a0"].data_ptr(), self.buf[0].data_ptr(),
-                                           self.buf[1].data_ptr(), self.nx, self.ny, self.nz,
-                                           d["c0"], d["c1"])
+                                           self.buf[1].data_ptr(), self.nx, self.ny, self.nz, d["c0"], d["c1"])
         grid = (_cdiv(self.nx, self.TX), _cdiv(self.ny, self.TY), _cdiv(self.nz, self.TZ))
         self.steps = [Step("stencil", grid, self.args, self.sweeps)]
 

@@ -63,6 +63,12 @@ class Accel:
         weights = [1] * len(jobs) if weights is None else weights
         fl = abi.REQ_LAUNCH_EVENTS if launch_events else 0
         reqs = [j.request(self.kids, t, e2e, w, fl) for j, t, w in zip(jobs, tenants, weights)]
+        # Job buffers (device inputs, tensor maps) were filled on torch's
+        # stream; libaccel launches on its own non-blocking streams, which do
+        # not order behind it.  Only torch's stream is waited on, never the
+        # device (requests already running keep running).
+        import torch
+        torch.cuda.current_stream(self.device).synchronize()
         return abi.accel_submit_group(self.ctx, reqs)
 
     def sync(self, rid: int = abi.ACCEL_ALL):
