@@ -151,6 +151,9 @@ typedef struct { void *dst; const void *src; uint64_t bytes; } accel_copy; /* ho
 /* accel_request.flags */
 #define ACCEL_REQ_LAUNCH_EVENTS 1u  /* record a CUDA event around every launch
                                        (per-launch device times via accel_launch_times) */
+#define ACCEL_REQ_TRACE 2u          /* record one accel_vg_record per virtual group
+                                       (accel_vg_trace); costs one %globaltimer
+                                       pair and a 24-B store per VG */
 
 typedef struct {
   int32_t tenant;             /* 0..ACCEL_MAX_TENANTS-1: selects the stream pair */
@@ -217,6 +220,19 @@ typedef struct {
 } accel_launch_stat;
 int accel_launch_stats(accel_ctx *ctx, uint64_t request_id, accel_launch_stat *out, uint32_t n,
                        uint32_t *n_out);
+/* Per-VG execution trace of a completed request submitted with
+ * ACCEL_REQ_TRACE (the tracing subsystem): record k of launch l
+ * of a step is at index (sum of the earlier launches' static VG totals) + k --
+ * the coverage layout.  t_start/t_end: %globaltimer around the body, sm =
+ * %smid, cta = the CTA (blockIdx.x of the persistent or top-up grid, linear
+ * block index of the native grid; top-up CTAs have bit 31 set).  VGs that did
+ * not run (bfs past the frontier) keep t_start_ns == 0.  n = capacity in
+ * records; *n_out = records of the request. */
+typedef struct {
+  uint64_t t_start_ns, t_end_ns;
+  uint32_t sm, cta;
+} accel_vg_record;
+int accel_vg_trace(accel_ctx *ctx, uint64_t request_id, accel_vg_record *out, uint64_t n, uint64_t *n_out);
 /* Forget completed requests (frees their descriptors); ACCEL_ALL = all done. */
 int accel_release(accel_ctx *ctx, uint64_t request_id);
 /* Streams of a tenant (cudaStream_t as void*), for interop (torch.cuda.ExternalStream). */

@@ -28,6 +28,7 @@ ACCEL_ALL = 2**64 - 1
 MAX_TENANTS = 16
 MAX_STEPS = 8
 REQ_LAUNCH_EVENTS = 1
+REQ_TRACE = 2
 
 u32, i32, u64, f32, f64, vp = C.c_uint32, C.c_int32, C.c_uint64, C.c_float, C.c_double, C.c_void_p
 
@@ -85,6 +86,10 @@ class accel_req_stats(C.Structure):
 class accel_launch_stat(C.Structure):
     _fields_ = [("t_first_ns", u64), ("t_last_ns", u64), ("ctas_started", u32), ("max_alive", u32),
                 ("total", u32), ("topped", u32)]
+
+
+class accel_vg_record(C.Structure):
+    _fields_ = [("t_start_ns", u64), ("t_end_ns", u64), ("sm", u32), ("cta", u32)]
 
 
 class accel_demand(C.Structure):
@@ -154,7 +159,7 @@ EXPORTS = [
     "accel_init", "accel_finalize", "accel_set_mode", "accel_last_error", "accel_builtin_kernel",
     "accel_builtin_count", "accel_builtin_name", "accel_kernel_register", "accel_kernel_info_get",
     "accel_submit", "accel_submit_group", "accel_sync", "accel_epoch", "accel_stats", "accel_release",
-    "accel_tenant_stream", "accel_launch_times", "accel_launch_stats", "accel_demand_of", "accel_solve", "accel_metrics", "accel_overlap", "accel_tma_map_2d",
+    "accel_tenant_stream", "accel_launch_times", "accel_launch_stats", "accel_vg_trace", "accel_demand_of", "accel_solve", "accel_metrics", "accel_overlap", "accel_tma_map_2d",
 ]
 
 
@@ -189,6 +194,7 @@ def _load() -> C.CDLL:
         "accel_tenant_stream": (i32, [vp, i32, P(vp), P(vp)]),
         "accel_launch_times": (i32, [vp, u64, P(f32), u32, P(u32)]),
         "accel_launch_stats": (i32, [vp, u64, P(accel_launch_stat), u32, P(u32)]),
+        "accel_vg_trace": (i32, [vp, u64, P(accel_vg_record), u64, P(u64)]),
         "accel_demand_of": (i32, [P(accel_caps), u32, u32, u32, u32, u32, P(accel_demand)]),
         "accel_solve": (i32, [P(accel_caps), P(accel_demand), i32, P(u32)]),
         "accel_metrics": (i32, [P(f64), P(f64), i32, P(accel_mix_metrics)]),
@@ -288,6 +294,18 @@ def accel_launch_stats(ctx, request_id: int, n: int) -> list[accel_launch_stat]:
     got = u32()
     check(lib.accel_launch_stats(ctx, request_id, buf, n, C.byref(got)), ctx)
     return list(buf)[:got.value]
+
+
+def accel_vg_trace(ctx, request_id: int):
+    """All VG records of a request submitted with REQ_TRACE, as a numpy
+    structured array (t_start_ns, t_end_ns, sm, cta)."""
+    import numpy as np
+    got = u64()
+    check(lib.accel_vg_trace(ctx, request_id, None, 0, C.byref(got)), ctx)
+    arr = np.zeros(got.value, dtype=[("t_start_ns", "<u8"), ("t_end_ns", "<u8"), ("sm", "<u4"), ("cta", "<u4")])
+    if got.value:
+        check(lib.accel_vg_trace(ctx, request_id, arr.ctypes.data_as(C.POINTER(accel_vg_record)), got.value, C.byref(got)), ctx)
+    return arr
 
 
 def accel_release(ctx, request_id: int = ACCEL_ALL) -> None:

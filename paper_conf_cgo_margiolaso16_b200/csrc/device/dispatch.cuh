@@ -39,6 +39,8 @@
 #include <cstdint>
 #include <type_traits>
 
+#include "accel.h"
+
 namespace accel {
 
 // Per-request control block (device memory).
@@ -66,7 +68,9 @@ struct alignas(128) Desc {
   Ctl* ctl;              // RESOLVE control block, nullptr otherwise
   uint32_t* coverage;    // verify: coverage[vg] += 1
   uint32_t has_prev;     // this - 1 is the request's previous launch
-  uint32_t pad0[19];
+  uint32_t pad_a;
+  accel_vg_record* trace;  // ACCEL_REQ_TRACE: trace[vg], nullptr otherwise
+  uint32_t pad0[16];
   // ---- line 1: the software queue head (RUN_TERMINATE when >= total)
   uint32_t next;
   uint32_t pad1[31];
@@ -114,6 +118,20 @@ __device__ __forceinline__ unsigned long long globaltimer() {
   asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
   return t;
 }
+__device__ __forceinline__ uint32_t smid() {
+  uint32_t v;
+  asm volatile("mov.u32 %0, %%smid;" : "=r"(v));
+  return v;
+}
+// ACCEL_REQ_TRACE: one record per VG, written by the master thread.
+__device__ __forceinline__ void trace_vg(accel_vg_record* t, uint32_t vg, unsigned long long t0, uint32_t cta) {
+  accel_vg_record r;
+  r.t_start_ns = t0;
+  r.t_end_ns = globaltimer();
+  r.sm = smid();
+  r.cta = cta;
+  t[vg] = r;
+}
 
 __device__ __forceinline__ uint32_t ld_relaxed(const uint32_t* p) {
   uint32_t v;
@@ -141,6 +159,27 @@ struct has_dynamic_total : std::false_type {};
 template <class T>
 struct has_dynamic_total<T, std::void_t<decltype(T::kDynamicTotal)>>
     : std::integral_constant<bool, T::kDynamicTotal> {};
+
+// kSpread: the kernel's VG cost varies smoothly in space (cutcp's atom
+// density, tpacf's pair blocks).  The CTAs of one SM reach the queue together,
+// so linear tickets hand each SM a run of adjacent -- equally heavy -- VGs and
+// the heavy runs pile up on a few SMs (issue-bound kernels then run 20 % long).
+// Spread kernels map ticket t -> VG t * p mod total (gcd(p, total) = 1,
+// p ~ total / golden ratio): consecutive tickets land far apart.
+template <class T, class = void>
+struct has_spread : std::false_type {};
+template <class T>
+struct has_spread<T, std::void_t<decltype(T::kSpread)>> : std::integral_constant<bool, T::kSpread> {};
+
+__device__ __forceinline__ uint32_t spread_factor(uint32_t total) {
+  if (total <= 2) return 1;
+  uint32_t p = (uint32_t)(0.6180339887 * total);
+  for (;; ++p) {
+    uint32_t a = p, b = total;
+    while (b) { const uint32_t r = a % b; a = b; b = r; }
+    if (a == 1) return p;
+  }
+}
 
 template <class T>
 __device__ __forceinline__ uint32_t vg_total(const typename T::Args& a, const Desc* d,
@@ -224,24 +263,57 @@ __device__ __forceinline__ bool admit(Desc* d) {
   return true;
 }
 
-// Per-CTA (thread 0) view of the live quota and the admitted count, loaded
-// right after each dequeue and used at the next one, so the RESOLVE check
-// adds no latency in front of the queue atomic.
-struct AdmHint {
-  uint32_t live = 0xffffffffu;
-  uint32_t alive = 0;
+// Scheduling state of one CTA in shared memory (the paper's `local struct SD`,
+// Fig. 8b).  Everything the master thread keeps between
+// dequeues lives here, not in registers, so the body keeps the register budget
+// it has in the native kernel: only the buffer parity k lives across the body.
+// The VG to run next is double-buffered: thread 0 publishes VG k+1 into
+// cur[(k+1)&1] while slower warps may still be loading cur[k&1] (a body
+// need not contain a barrier); the barrier closing iteration k orders both.
+struct SchedState {
+  struct Cur {
+    uint32_t vg;         // queue position to run next (sd.wg_base)
+    uint32_t id;         // the VG at that position (vg, or spread)
+    uint32_t x, y, z;    // its decode, by thread 0 (the warps only load it)
+  } cur[2];
+  uint32_t end;        // end of the current chunk (sd.wg_end)
+  uint32_t total;      // VGs of this launch (RUN_TERMINATE when vg >= total)
+  uint32_t gx, gy, gz, launch_idx;
+  uint32_t spread;     // 0: linear, else the kSpread factor
+  uint32_t chunk;
+  uint32_t prefetch_window;
+  uint32_t nxt;        // prefetched chunk (valid if have_nxt)
+  uint32_t* coverage;
+  accel_vg_record* trace;
+  unsigned long long t0;   // trace: start of the current VG
+  // RESOLVE, thread 0: view of the live quota and the admitted count, loaded
+  // right after each dequeue and used at the next one, so the check adds no
+  // latency in front of the queue atomic
+  uint32_t hint_live, hint_alive;
+  uint8_t have_nxt, admitted, draining;
+  uint8_t long_vg;     // the last VG ran longer than kLongVgNs
+  template <bool kSpread>
+  __device__ __forceinline__ void set_cur(uint32_t k, uint32_t vg) {
+    cur[k].vg = vg;
+    if (vg < total) {
+      uint32_t id = vg;
+      if constexpr (kSpread) id = (uint32_t)(((uint64_t)vg * spread) % total);
+      cur[k].id = id;
+      const VirtualBlock b = decode(id, gx, gy, gz, launch_idx);
+      cur[k].x = b.x; cur[k].y = b.y; cur[k].z = b.z;
+    }
+  }
 };
 
 // One dequeue (Fig. 8b line 26, rt_sched_wgroup): under RESOLVE a CTA
 // leaves first if the launch holds more CTAs than the live quota (shrink at a
 // VG boundary; CAS so exactly alive - live CTAs leave); then one atomicAdd of
-// `chunk` on the queue head.  The dequeue is a prefetch issued while the CTA's
-// current VG is still running, so an evicted CTA is `draining` (counted by
-// wait_complete) until retire(), after that VG's results are written.
+// `chunk` on the queue head.  The dequeue may be a prefetch issued while the
+// CTA's current VG is still running, so an evicted CTA is `draining` (counted
+// by wait_complete) until retire(), after that VG's results are written.
 template <bool kResolve>
-__device__ __forceinline__ uint32_t dequeue(Desc* d, uint32_t chunk, bool& admitted, bool& draining,
-                                            AdmHint& hint) {
-  if (kResolve && hint.alive > hint.live) {
+__device__ __forceinline__ uint32_t dequeue(Desc* d, SchedState* S) {
+  if (kResolve && S->hint_alive > S->hint_live) {
     uint32_t live = ld_relaxed(&d->ctl->live);
     uint32_t a = ld_relaxed(&d->alive);
     if (a > live) {
@@ -252,8 +324,8 @@ __device__ __forceinline__ uint32_t dequeue(Desc* d, uint32_t chunk, bool& admit
         if (prev == a) {
           red_add_u32(&d->adm, 0xffffffffu);
           red_add_u32(&d->evicted, 1u);
-          admitted = false;
-          draining = true;
+          S->admitted = 0;
+          S->draining = 1;
           return kTerminate;
         }
         a = prev;
@@ -261,62 +333,36 @@ __device__ __forceinline__ uint32_t dequeue(Desc* d, uint32_t chunk, bool& admit
       red_add_u32(&d->draining, 0xffffffffu);   // not evicted after all
     }
   }
-  const uint32_t b = atomicAdd(&d->next, chunk);
+  const uint32_t b = atomicAdd(&d->next, S->chunk);
   if (kResolve) {
-    hint.live = ld_relaxed(&d->ctl->live);
-    hint.alive = ld_relaxed(&d->alive);
+    S->hint_live = ld_relaxed(&d->ctl->live);
+    S->hint_alive = ld_relaxed(&d->alive);
   }
   return b;
 }
 
 template <bool kResolve>
-__device__ __forceinline__ void retire(Desc* d, uint32_t cfg, bool admitted, bool draining) {
-  if (kResolve && admitted) {
+__device__ __forceinline__ void retire(Desc* d, uint32_t cfg, const SchedState* S) {
+  if (kResolve && S->admitted) {
     __threadfence();  // this CTA's VG results before the alive decrement
     atomicSub(&d->alive, 1u);
     red_add_u32(&d->adm, 0xffffffffu);
   }
-  if (kResolve && draining) {
+  if (kResolve && S->draining) {
     __threadfence();  // the last VG's results before the draining decrement
     atomicSub(&d->draining, 1u);
   }
   if (cfg & kCfgStamps) red_max_u64(&d->t_last, globaltimer());
 }
 
-// Scheduling state of one CTA in shared memory (the paper's `local struct SD`,
-// Fig. 8b).  Keeping it in shared memory instead of registers
-// leaves the body the same register budget it has in the native kernel: only
-// the current VG id and the prefetched chunk id live across the body call.
-// The VG to run next is double-buffered: thread 0 publishes VG k+1 into
-// cur[(k+1)&1] while slower warps may still be loading cur[k&1] (a body
-// need not contain a barrier); the barrier closing iteration k orders both.
-struct SchedState {
-  struct Cur {
-    uint32_t vg;         // VG to run next (sd.wg_base)
-    uint32_t x, y, z;    // its decode, by thread 0 (the warps only load it)
-  } cur[2];
-  uint32_t end;        // end of the current chunk (sd.wg_end)
-  uint32_t total;      // VGs of this launch (RUN_TERMINATE when vg >= total)
-  uint32_t gx, gy, gz, launch_idx;
-  uint32_t* coverage;
-  __device__ __forceinline__ void set_cur(uint32_t k, uint32_t vg) {
-    cur[k].vg = vg;
-    if (vg < total) {
-      const VirtualBlock b = decode(vg, gx, gy, gz, launch_idx);
-      cur[k].x = b.x; cur[k].y = b.y; cur[k].z = b.z;
-    }
-  }
-};
+constexpr unsigned long long kLongVgNs = 40000;   // 40 us: ~20 queue round trips
 
 // Serve one launch: admission, dequeue loop, retire.  All threads call it.
 template <class T, bool kResolve>
 __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, char* smem,
-                                      SchedState* S, uint32_t cfg) {
-  const uint32_t chunk = cfg & kCfgChunkMask;
-  bool admitted = true;      // meaningful in thread 0 only
-  bool draining = false;     // thread 0: evicted at the prefetch, last VG in flight
-  AdmHint hint;              // thread 0, RESOLVE only
+                                      SchedState* S, uint32_t cfg, uint32_t cta_tag) {
   if (threadIdx.x == 0) {    // master work-item: environment init (rt_env_init)
+    const uint32_t chunk = cfg & kCfgChunkMask;
     uint32_t b = kTerminate;
     // STATIC: the first dequeue is issued before anything else is loaded
     if (!kResolve) b = atomicAdd(&d->next, chunk);
@@ -324,10 +370,17 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     const uint32_t launch_idx = d->launch_idx;
     const uint32_t total = vg_total<T>(args, d, launch_idx);
     if (blockIdx.x == 0) d->total_seen = total;
+    S->chunk = chunk;
+    S->admitted = 1;
+    S->draining = 0;
+    S->have_nxt = 0;
+    S->long_vg = 0;
+    S->hint_live = 0xffffffffu;
+    S->hint_alive = 0;
     if (kResolve) {
       asm volatile("red.relaxed.gpu.global.max.u32 [%0], %1;" ::"l"(&d->ctl->cur), "r"(d->req_idx) : "memory");
-      admitted = admit(d);
-      if (admitted) b = dequeue<true>(d, chunk, admitted, draining, hint);
+      S->admitted = admit(d) ? 1 : 0;
+      if (S->admitted) b = dequeue<true>(d, S);
     }
     if (b < total) red_add_u32(&d->ctas_started, 1u);
     S->end = b < total ? min(b + chunk, total) : b;
@@ -337,39 +390,51 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     S->gz = d->gz;
     S->launch_idx = launch_idx;
     S->coverage = d->coverage;
-    S->set_cur(0, b);
+    S->trace = d->trace;
+    S->spread = has_spread<T>::value ? spread_factor(total) : 0u;
+    S->prefetch_window = 2u * chunk * gridDim.x;
+    S->template set_cur<has_spread<T>::value>(0, b);
   }
   __syncthreads();
-  uint32_t nxt = kTerminate;  // thread 0: id of the next chunk, requested at chunk start
-  bool have_nxt = false;
   for (uint32_t k = 0;; k ^= 1u) {
     const SchedState::Cur c = S->cur[k];
-    const uint32_t vg = c.vg;
-    if (vg >= S->total) break;                 // RUN_TERMINATE
-    if (threadIdx.x == 0 && !have_nxt) {
-      // prefetch the next chunk id once per chunk, early (hidden behind the body)
-      nxt = dequeue<kResolve>(d, chunk, admitted, draining, hint);
-      have_nxt = true;
+    if (c.vg >= S->total) break;                 // RUN_TERMINATE
+    if (threadIdx.x == 0) {
+      if (!S->have_nxt && (!S->long_vg || S->total - S->end > S->prefetch_window)) {
+        // prefetch the next chunk id once per chunk, early (hidden behind the
+        // body).  A prefetched id is a reservation: in the last waves,
+        // reservations held by busy CTAs leave finished CTAs (whole SMs) idle
+        // for up to one VG duration.  So kernels whose VGs run long (where
+        // that idle time dwarfs one queue round trip) dequeue just in time
+        // once fewer than two waves of VGs remain
+        S->nxt = dequeue<kResolve>(d, S);
+        S->have_nxt = 1;
+      }
+      S->t0 = globaltimer();
     }
     VirtualBlock vb;
     vb.x = c.x; vb.y = c.y; vb.z = c.z;
     vb.gx = S->gx; vb.gy = S->gy; vb.gz = S->gz;
-    vb.linear = vg;
+    vb.linear = c.id;
     vb.launch_idx = S->launch_idx;
     T::body(args, vb, smem);
     if (threadIdx.x == 0) {
-      if (S->coverage != nullptr) atomicAdd(&S->coverage[vg], 1u);
+      const uint32_t vg = S->cur[k].vg, id = S->cur[k].id;
+      if (S->coverage != nullptr) atomicAdd(&S->coverage[id], 1u);
+      if (S->trace != nullptr) trace_vg(S->trace, id, S->t0, cta_tag);
+      S->long_vg = globaltimer() - S->t0 > kLongVgNs;
       if (vg + 1 < S->end) {
-        S->set_cur(k ^ 1u, vg + 1);
+        S->template set_cur<has_spread<T>::value>(k ^ 1u, vg + 1);
       } else {                                   // publish the prefetched chunk
-        S->end = nxt < S->total ? min(nxt + chunk, S->total) : nxt;
-        S->set_cur(k ^ 1u, nxt);
-        have_nxt = false;
+        const uint32_t nxt = S->have_nxt ? S->nxt : dequeue<kResolve>(d, S);   // tail: just in time
+        S->end = nxt < S->total ? min(nxt + S->chunk, S->total) : nxt;
+        S->template set_cur<has_spread<T>::value>(k ^ 1u, nxt);
+        S->have_nxt = 0;
       }
     }
     __syncthreads();
   }
-  if (threadIdx.x == 0) retire<kResolve>(d, cfg, admitted, draining);
+  if (threadIdx.x == 0) retire<kResolve>(d, cfg, S);
 }
 
 // -------------------------------------------------------------------------
@@ -384,7 +449,7 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
     if (threadIdx.x == 0 && d->has_prev && ld_volatile(&(d - 1)->topped)) wait_complete(d - 1);
     __syncthreads();
   }
-  serve<T, kResolve>(args, d, smem, &S, cfg);
+  serve<T, kResolve>(args, d, smem, &S, cfg, blockIdx.x);
 }
 
 // RESOLVE top-up grid: d = first launch of the request step, `sticky` =
@@ -410,7 +475,7 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
     }
     __syncthreads();
     const uint32_t cfg = dl->chunk | kCfgResolve | ((dl->flags & kFlagStamps) ? kCfgStamps : 0u);
-    serve<T, true>(args, dl, smem, &S, cfg);
+    serve<T, true>(args, dl, smem, &S, cfg, blockIdx.x | 0x80000000u);
     __syncthreads();
   }
 }
@@ -435,8 +500,13 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
   }
   if (vb.linear == 0 && threadIdx.x == 0) d->total_seen = total;
   if (run) {
+    __shared__ unsigned long long s_t0;   // trace: thread 0's VG start (not a register across the body)
+    if (threadIdx.x == 0 && d->trace != nullptr) s_t0 = globaltimer();
     T::body(args, vb, smem);
-    if (d->coverage != nullptr && threadIdx.x == 0) atomicAdd(&d->coverage[vb.linear], 1u);
+    if (threadIdx.x == 0) {
+      if (d->coverage != nullptr) atomicAdd(&d->coverage[vb.linear], 1u);
+      if (d->trace != nullptr) trace_vg(d->trace, vb.linear, s_t0, vb.linear);
+    }
   }
   if (threadIdx.x == 0 && (flags & kFlagStamps)) red_max_u64(&d->t_last, globaltimer());
 }

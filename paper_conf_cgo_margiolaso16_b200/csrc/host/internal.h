@@ -25,6 +25,7 @@ struct InitParams {
   Ctl* ctl;               // RESOLVE control block, nullptr under STATIC
   uint32_t live_init;     // initial live quota of the main step
   uint32_t* coverage;     // nullptr unless verify
+  accel_vg_record* trace; // nullptr unless ACCEL_REQ_TRACE
   uint32_t flags;
   uint32_t n_steps;
   InitStep steps[ACCEL_MAX_STEPS];

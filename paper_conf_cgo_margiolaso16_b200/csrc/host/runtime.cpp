@@ -81,6 +81,8 @@ struct Request {
   uint32_t slot = 0, n_desc = 0;
   uint32_t* cov = nullptr;
   uint64_t cov_elems = 0;
+  accel_vg_record* trace = nullptr;   // ACCEL_REQ_TRACE, cov layout
+  uint64_t trace_elems = 0;
   uint32_t quota_initial = 0, quota_min = 0, quota_max = 0, resolves = 0;
   uint32_t live = 0;         // RESOLVE: current live quota of the main step
   uint32_t provisioned = 0;  // RESOLVE: main-grid CTAs + sticky top-up CTAs
@@ -116,7 +118,9 @@ struct DescHost {
   // line 0
   uint32_t total, gx, gy, gz, chunk, launch_idx, flags, req_idx;
   uint64_t ctl, coverage;
-  uint32_t has_prev, pad0[19];
+  uint32_t has_prev, pad_a;
+  uint64_t trace;
+  uint32_t pad0[16];
   // line 1
   uint32_t next, pad1[31];
   // line 2
@@ -274,12 +278,14 @@ int enqueue(accel_ctx* ctx, Request* r) {
   for (const accel_clear& c : r->clears) CK(ctx, cudaMemsetAsync(c.dst_device, c.value, c.bytes, s));
   for (const accel_copy& c : r->h2d) CK(ctx, cudaMemcpyAsync(c.dst, c.src, c.bytes, cudaMemcpyHostToDevice, s));
   if (r->cov) CK(ctx, cudaMemsetAsync(r->cov, 0, r->cov_elems * sizeof(uint32_t), s));
+  if (r->trace) CK(ctx, cudaMemsetAsync(r->trace, 0, r->trace_elems * sizeof(accel_vg_record), s));
   InitParams p{};
   p.d = ctx->desc_ptr(r->slot);
   const bool resolve = shared && ctx->cfg.policy == ACCEL_POLICY_RESOLVE;
   p.ctl = resolve ? ctx->ctl_ptr(r->slot) : nullptr;
   p.live_init = r->steps[r->main_step].quota;
   p.coverage = r->cov;
+  p.trace = r->trace;
   p.flags = kFlagStamps | (shared ? kFlagAlive : 0u);
   p.n_steps = (uint32_t)r->steps.size();
   for (size_t j = 0; j < r->steps.size(); ++j) {
@@ -353,6 +359,7 @@ int build_request(accel_ctx* ctx, const accel_request& in, std::unique_ptr<Reque
   }
   r->n_desc = n_desc;
   r->cov_elems = ctx->cfg.verify ? cov : 0;
+  r->trace_elems = (in.flags & ACCEL_REQ_TRACE) ? cov : 0;
   r->clears.assign(in.clear, in.clear + in.n_clear);
   r->h2d.assign(in.h2d, in.h2d + in.n_h2d);
   r->d2h.assign(in.d2h, in.d2h + in.n_d2h);
@@ -446,6 +453,13 @@ int assign_quotas(accel_ctx* ctx, std::vector<std::unique_ptr<Request>>& fresh) 
         s.quota = qj[i];
       }
     }
+    if (const char* e = std::getenv("ACCEL_QUOTA_MULT")) {
+      // experiment knob (scripts/vg_trace.py): oversubscribe every step's grid
+      // by a factor, e.g. a multiple large enough for one VG per CTA
+      const double m = std::atof(e);
+      for (Step& s : r->steps) s.quota = (uint32_t)std::min<double>(s.total, std::max(1.0, s.quota * m));
+      q[i] = r->steps[r->main_step].quota;
+    }
     r->quota_initial = r->quota_min = r->quota_max = q[i];
     r->live = r->provisioned = q[i];
   }
@@ -508,6 +522,7 @@ int submit_locked(accel_ctx* ctx, uint32_t n, const accel_request* rs, uint64_t*
     }
     r->slot = (uint32_t)s;
     if (r->cov_elems) CK(ctx, cudaMalloc(&r->cov, r->cov_elems * sizeof(uint32_t)));
+    if (r->trace_elems) CK(ctx, cudaMalloc(&r->trace, r->trace_elems * sizeof(accel_vg_record)));
   }
   for (uint32_t i = 0; i < n; ++i) {
     Request* r = fresh[i].get();
@@ -523,6 +538,7 @@ int submit_locked(accel_ctx* ctx, uint32_t n, const accel_request* rs, uint64_t*
 void release_request(accel_ctx* ctx, Request* r) {
   ctx->free_slots(r->slot, r->n_desc);
   if (r->cov) cudaFree(r->cov);
+  if (r->trace) cudaFree(r->trace);
   if (r->ev_arrival) ctx->free_events.push_back(r->ev_arrival);
   if (r->ev_done) ctx->free_events.push_back(r->ev_done);
   for (cudaEvent_t ev : r->ev_launch) ctx->free_events.push_back(ev);
@@ -841,6 +857,23 @@ int accel_launch_stats(accel_ctx* ctx, uint64_t request_id, accel_launch_stat* o
     out[i].topped = d->topped;
   }
   *n_out = m;
+  return ACCEL_OK;
+}
+
+int accel_vg_trace(accel_ctx* ctx, uint64_t request_id, accel_vg_record* out, uint64_t n, uint64_t* n_out) {
+  if (!ctx || (n && !out) || !n_out) return ACCEL_EINVAL;
+  std::lock_guard<std::mutex> g(ctx->mu);
+  if (ctx->poisoned) return ACCEL_ESTATE;
+  auto it = ctx->reqs.find(request_id);
+  if (it == ctx->reqs.end()) return ctx->fail(ACCEL_EINVAL, "unknown request");
+  Request* r = it->second.get();
+  if (!r->trace) return ctx->fail(ACCEL_EINVAL, "request was not submitted with ACCEL_REQ_TRACE");
+  int rc = refresh_done(ctx, r);
+  if (rc) return rc;
+  if (!r->done) return ACCEL_ENOTREADY;
+  const uint64_t m = std::min<uint64_t>(n, r->trace_elems);
+  if (m) CK(ctx, cudaMemcpy(out, r->trace, m * sizeof(accel_vg_record), cudaMemcpyDeviceToHost));
+  *n_out = r->trace_elems;
   return ACCEL_OK;
 }
 

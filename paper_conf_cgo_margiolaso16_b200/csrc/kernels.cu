@@ -45,6 +45,7 @@ __global__ void desc_init_kernel(const InitParams p, uint32_t n_desc) {
   d->total_seen = kTerminate;
   d->ctl = p.ctl;
   d->coverage = p.coverage ? p.coverage + st.cov_offset + (size_t)r * st.total : nullptr;
+  d->trace = p.trace ? p.trace + st.cov_offset + (size_t)r * st.total : nullptr;
   d->t_first = ULLONG_MAX;
   d->t_last = 0;
   d->ctas_started = 0;

@@ -31,13 +31,13 @@ struct Stencil {
   static constexpr int kThreads = 256;
   static constexpr int kTX = 128, kTY = 8, kTZ = 8;
   static constexpr uint32_t kChunk = 1;
-  static constexpr int kMinBlocks = 6;
+  static constexpr int kMinBlocks = 5;
   static constexpr int kRows = kTY + 2;                 // y halo
   static constexpr int kCols = kTX + 8;                 // x0-4 .. x0+131 (16-B multiples)
   static constexpr uint32_t kPlaneBytes = kRows * kCols * 4;          // 5440
   static constexpr uint32_t kSlot = (kPlaneBytes + 127) / 128 * 128;  // 5504
 #ifndef STENCIL_KD
-#define STENCIL_KD 3
+#define STENCIL_KD 4
 #endif
   static constexpr int kD = STENCIL_KD;                 // planes in flight beyond z+1
   static constexpr int kR = kD + 2;                     // ring slots

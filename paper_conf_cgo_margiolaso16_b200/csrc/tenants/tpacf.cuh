@@ -20,6 +20,7 @@ struct Tpacf {
   using Args = accel_tpacf_args;
   static constexpr int kThreads = 256;
   static constexpr uint32_t kChunk = 1;
+  static constexpr bool kSpread = true;     // VG cost varies in space (dispatch.cuh)
   static constexpr int kMinBlocks = 6;   // <= 40 regs: smem allows 6 CTAs/SM
   static constexpr int kWarps = kThreads / 32;
   static constexpr int kMaxBins = 32;      // nedges + 1 <= 32

@@ -57,11 +57,12 @@ class Accel:
         return abi.accel_kernel_info_get(self.ctx, self.kids[name])
 
     def submit(self, jobs: list[Job], tenants: list[int] | None = None, e2e: bool = False,
-               weights: list[int] | None = None, launch_events: bool = False) -> list[int]:
-        """Submit jobs as one group arriving together, in list order."""
+               weights: list[int] | None = None, launch_events: bool = False, trace: bool = False) -> list[int]:
+        """Submit jobs as one group arriving together, in list order.
+        trace: record every virtual group (vg_trace)."""
         tenants = list(range(len(jobs))) if tenants is None else tenants
         weights = [1] * len(jobs) if weights is None else weights
-        fl = abi.REQ_LAUNCH_EVENTS if launch_events else 0
+        fl = (abi.REQ_LAUNCH_EVENTS if launch_events else 0) | (abi.REQ_TRACE if trace else 0)
         reqs = [j.request(self.kids, t, e2e, w, fl) for j, t, w in zip(jobs, tenants, weights)]
         # Job buffers (device inputs, tensor maps) were filled on torch's
         # stream; libaccel launches on its own non-blocking streams, which do
@@ -85,6 +86,10 @@ class Accel:
 
     def launch_times(self, rid: int, n: int) -> list[float]:
         return abi.accel_launch_times(self.ctx, rid, n)
+
+    def vg_trace(self, rid: int):
+        """Per-VG records (t_start_ns, t_end_ns, sm, cta) of a traced request."""
+        return abi.accel_vg_trace(self.ctx, rid)
 
     def release(self, rid: int = abi.ACCEL_ALL):
         abi.accel_release(self.ctx, rid)
