@@ -28,7 +28,9 @@
 // request's live quota lives in a device control word.  Admission is
 // count-based: a CTA works on a launch only while that launch's `alive` count
 // is <= live, so shrinking takes effect at the next dequeue of every CTA
-// (a VG boundary), and growing adds CTAs -- sticky top-up grids launched by the
+// (a VG boundary).  `alive` shares one 64-bit word with the queue head, so
+// admission and the first dequeue are ONE atomic (and every dequeue returns a
+// fresh alive count for free).  Growing adds CTAs -- sticky top-up grids launched by the
 // host monitor on the tenant's second stream, which serve the current launch
 // and then follow the request's later launches.  Because a top-up CTA may
 // still run VGs of launch l after launch l's main grid retired, a launch whose
@@ -70,22 +72,26 @@ struct alignas(128) Desc {
   uint32_t has_prev;     // this - 1 is the request's previous launch
   uint32_t pad_a;
   accel_vg_record* trace;  // ACCEL_REQ_TRACE: trace[vg], nullptr otherwise
-  uint32_t pad0[16];
-  // ---- line 1: the software queue head (RUN_TERMINATE when >= total)
-  uint32_t next;
-  uint32_t pad1[31];
+  uint32_t governed;       // RESOLVE: this launch belongs to the request's main
+                           // step, whose CTA count the live quota governs (the
+                           // other steps keep their own solved grid)
+  uint32_t pad0[15];
+  // ---- line 1: the software queue head (RUN_TERMINATE when >= total) in the
+  // low 32 bits, the admitted CTA count (`alive`, RESOLVE) in the high 32
+  unsigned long long qa;
+  uint32_t pad1[30];
   // ---- line 2
   unsigned long long t_first;  // min %globaltimer over CTA starts
   unsigned long long t_last;   // max %globaltimer over CTA ends
   uint32_t total_seen;   // total as read by the CTAs (dynamic for bfs)
   uint32_t ctas_started; // CTAs admitted with work
-  uint32_t alive;        // CTAs currently admitted (RESOLVE)
+  uint32_t pad_alive;
   uint32_t max_alive;    // high-water mark of `alive` (RESOLVE)
   uint32_t topped;       // a top-up CTA joined this launch (RESOLVE)
-  uint32_t admit_fail;   // RESOLVE: CTAs refused at admission
+  uint32_t admit_fail;   // RESOLVE: CTAs admitted over the live quota (ran one chunk, left)
   uint32_t evicted;      // RESOLVE: CTAs that left at a dequeue (shrink)
   uint32_t last_live;    // RESOLVE: live quota seen by the last refused CTA
-  uint32_t adm;          // RESOLVE: admission tickets (alive + in-flight refusals)
+  uint32_t pad_adm;
   uint32_t draining;     // RESOLVE: evicted CTAs still finishing their last VG
   uint32_t pad2[18];
 };
@@ -103,6 +109,12 @@ __device__ __forceinline__ void red_add_u32(uint32_t* p, uint32_t v) {
 }
 
 enum : uint32_t { kFlagStamps = 1u, kFlagAlive = 2u };
+
+// Desc::qa = alive << 32 | next
+constexpr unsigned long long kAlive1 = 1ull << 32;
+constexpr unsigned long long kAliveNeg = ~0ull << 32;   // adds -1 to the alive half
+__device__ __forceinline__ uint32_t qa_next(unsigned long long v) { return (uint32_t)v; }
+__device__ __forceinline__ uint32_t qa_alive(unsigned long long v) { return (uint32_t)(v >> 32); }
 
 // Replacement of the OpenCL work-item built-ins (get_group_id / get_num_groups,
 // PAPER.md §6.3): what a body sees instead of blockIdx/gridDim.
@@ -142,6 +154,15 @@ __device__ __forceinline__ uint32_t ld_relaxed(const uint32_t* p) {
 __device__ __forceinline__ uint32_t ld_volatile(const uint32_t* p) {
   uint32_t v;
   asm volatile("ld.volatile.global.u32 %0, [%1];" : "=r"(v) : "l"(p));
+  return v;
+}
+// Release/acquire fence at GPU scope (message passing between CTAs); lighter
+// than __threadfence() (fence.sc.gpu).
+__device__ __forceinline__ void fence_acq_rel() { asm volatile("fence.acq_rel.gpu;" ::: "memory"); }
+
+__device__ __forceinline__ unsigned long long ld_volatile_u64(const unsigned long long* p) {
+  unsigned long long v;
+  asm volatile("ld.volatile.global.u64 %0, [%1];" : "=l"(v) : "l"(p));
   return v;
 }
 
@@ -216,16 +237,14 @@ constexpr uint32_t kTerminate = 0xffffffffu;
 __device__ __forceinline__ void wait_complete(const Desc* p) {
   for (;;) {
     const uint32_t tot = ld_volatile(&p->total_seen);
-    if (tot != kTerminate && ld_volatile(&p->next) >= tot) {
-      __threadfence();
-      if (ld_volatile(&p->alive) == 0) {
-        __threadfence();
-        if (ld_volatile(&p->draining) == 0) break;
-      }
+    const unsigned long long v = ld_volatile_u64(&p->qa);
+    if (tot != kTerminate && qa_next(v) >= tot && qa_alive(v) == 0) {
+      fence_acq_rel();
+      if (ld_volatile(&p->draining) == 0) break;
     }
     __nanosleep(256);
   }
-  __threadfence();
+  fence_acq_rel();
   // the launch's results were written through the generic proxy by other CTAs;
   // this CTA may read them with TMA (async proxy)
   asm volatile("fence.proxy.async.global;" ::: "memory");
@@ -240,28 +259,6 @@ enum : uint32_t {
   kCfgResolve = 1u << 16,
   kCfgStamps = 1u << 17
 };
-
-// Master work-item, admission into launch d under RESOLVE (count-based).
-// Two counters: `adm` hands out tickets (a refused CTA gives its ticket back,
-// so adm can be transiently high -- at worst a concurrent arrival is refused
-// spuriously), `alive` counts admitted CTAs exactly and is what eviction
-// reads (an atomicAdd/atomicSub pair on `alive` itself made admitted CTAs see a
-// transient alive > live and evict themselves; a CAS loop on it serialised
-// hundreds of CTAs at every launch start).
-__device__ __forceinline__ bool admit(Desc* d) {
-  const uint32_t live = ld_relaxed(&d->ctl->live);
-  const uint32_t t = atomicAdd(&d->adm, 1u);
-  if (t >= live) {
-    red_add_u32(&d->adm, 0xffffffffu);   // -1
-    red_add_u32(&d->admit_fail, 1u);
-    d->last_live = live;
-    return false;
-  }
-  const uint32_t a = atomicAdd(&d->alive, 1u) + 1u;
-  asm volatile("red.relaxed.gpu.global.max.u32 [%0], %1;" ::"l"(&d->max_alive), "r"(a) : "memory");
-  __threadfence();  // admission visible before the first dequeue
-  return true;
-}
 
 // Scheduling state of one CTA in shared memory (the paper's `local struct SD`,
 // Fig. 8b).  Everything the master thread keeps between
@@ -291,6 +288,7 @@ struct SchedState {
   // latency in front of the queue atomic
   uint32_t hint_live, hint_alive;
   uint8_t have_nxt, admitted, draining;
+  uint8_t over;        // RESOLVE: admitted over the live quota -> leave at the next dequeue
   uint8_t long_vg;     // the last VG ran longer than kLongVgNs
   template <bool kSpread>
   __device__ __forceinline__ void set_cur(uint32_t k, uint32_t vg) {
@@ -305,51 +303,53 @@ struct SchedState {
   }
 };
 
-// One dequeue (Fig. 8b line 26, rt_sched_wgroup): under RESOLVE a CTA
-// leaves first if the launch holds more CTAs than the live quota (shrink at a
-// VG boundary; CAS so exactly alive - live CTAs leave); then one atomicAdd of
-// `chunk` on the queue head.  The dequeue may be a prefetch issued while the
-// CTA's current VG is still running, so an evicted CTA is `draining` (counted
-// by wait_complete) until retire(), after that VG's results are written.
+// One dequeue (Fig. 8b line 26, rt_sched_wgroup): one 64-bit
+// atomicAdd of `chunk` on the queue word, which also returns the admitted
+// count.  Under RESOLVE a CTA first leaves if its last view says the launch
+// holds more CTAs than the live quota (shrink at a VG boundary; a CAS on the
+// alive half so exactly alive - live CTAs leave), or if it was admitted over
+// the quota.  A dequeue may be a prefetch issued while the CTA's current VG is
+// still running, so an evicted CTA is `draining` (counted by wait_complete)
+// until retire(), after that VG's results are written.  Returns the raw queue
+// word (kEvicted when the CTA left).
+constexpr unsigned long long kEvicted = ~0ull;
 template <bool kResolve>
-__device__ __forceinline__ uint32_t dequeue(Desc* d, SchedState* S) {
-  if (kResolve && S->hint_alive > S->hint_live) {
-    uint32_t live = ld_relaxed(&d->ctl->live);
-    uint32_t a = ld_relaxed(&d->alive);
-    if (a > live) {
-      atomicAdd(&d->draining, 1u);
-      __threadfence();   // draining visible before alive drops
-      while (a > live) {
-        const uint32_t prev = atomicCAS(&d->alive, a, a - 1u);
-        if (prev == a) {
-          red_add_u32(&d->adm, 0xffffffffu);
-          red_add_u32(&d->evicted, 1u);
-          S->admitted = 0;
-          S->draining = 1;
-          return kTerminate;
-        }
-        a = prev;
+__device__ __forceinline__ unsigned long long dequeue(Desc* d, SchedState* S) {
+  if (kResolve && (S->over || S->hint_alive > S->hint_live)) {
+    atomicAdd(&d->draining, 1u);
+    fence_acq_rel();   // draining visible before alive drops
+    bool left = false;
+    if (S->over) {
+      atomicAdd(&d->qa, kAliveNeg);
+      left = true;
+    } else {
+      const uint32_t live = ld_relaxed(&d->ctl->live);
+      unsigned long long v = ld_volatile_u64(&d->qa);
+      while (qa_alive(v) > live) {
+        const unsigned long long prev = atomicCAS(&d->qa, v, v + kAliveNeg);
+        if (prev == v) { left = true; break; }
+        v = prev;
       }
-      red_add_u32(&d->draining, 0xffffffffu);   // not evicted after all
     }
+    if (left) {
+      red_add_u32(&d->evicted, 1u);
+      S->admitted = 0;
+      S->draining = 1;
+      return kEvicted;
+    }
+    red_add_u32(&d->draining, 0xffffffffu);   // not evicted after all
   }
-  const uint32_t b = atomicAdd(&d->next, S->chunk);
-  if (kResolve) {
-    S->hint_live = ld_relaxed(&d->ctl->live);
-    S->hint_alive = ld_relaxed(&d->alive);
-  }
-  return b;
+  return atomicAdd(&d->qa, (unsigned long long)S->chunk);
 }
 
 template <bool kResolve>
 __device__ __forceinline__ void retire(Desc* d, uint32_t cfg, const SchedState* S) {
   if (kResolve && S->admitted) {
-    __threadfence();  // this CTA's VG results before the alive decrement
-    atomicSub(&d->alive, 1u);
-    red_add_u32(&d->adm, 0xffffffffu);
+    fence_acq_rel();  // this CTA's VG results before the alive decrement
+    atomicAdd(&d->qa, kAliveNeg);
   }
   if (kResolve && S->draining) {
-    __threadfence();  // the last VG's results before the draining decrement
+    fence_acq_rel();  // the last VG's results before the draining decrement
     atomicSub(&d->draining, 1u);
   }
   if (cfg & kCfgStamps) red_max_u64(&d->t_last, globaltimer());
@@ -363,25 +363,36 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
                                       SchedState* S, uint32_t cfg, uint32_t cta_tag) {
   if (threadIdx.x == 0) {    // master work-item: environment init (rt_env_init)
     const uint32_t chunk = cfg & kCfgChunkMask;
-    uint32_t b = kTerminate;
-    // STATIC: the first dequeue is issued before anything else is loaded
-    if (!kResolve) b = atomicAdd(&d->next, chunk);
+    uint32_t b;
+    S->admitted = 1;
+    S->draining = 0;
+    S->over = 0;
+    if (!kResolve) {
+      b = qa_next(atomicAdd(&d->qa, (unsigned long long)chunk));   // issued before anything else
+    } else {
+      // admission and first dequeue in one atomic; an arrival over the live
+      // quota runs the chunk it got and leaves at its next dequeue
+      asm volatile("red.relaxed.gpu.global.max.u32 [%0], %1;" ::"l"(&d->ctl->cur), "r"(d->req_idx) : "memory");
+      const uint32_t live = d->governed ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
+      const unsigned long long v = atomicAdd(&d->qa, kAlive1 | chunk);
+      b = qa_next(v);
+      const uint32_t a = qa_alive(v) + 1u;
+      asm volatile("red.relaxed.gpu.global.max.u32 [%0], %1;" ::"l"(&d->max_alive), "r"(a) : "memory");
+      if (a > live) {
+        S->over = 1;
+        red_add_u32(&d->admit_fail, 1u);
+        d->last_live = live;
+      }
+      S->hint_live = live;
+      S->hint_alive = a;
+    }
     if (cfg & kCfgStamps) red_min_u64(&d->t_first, globaltimer());
     const uint32_t launch_idx = d->launch_idx;
     const uint32_t total = vg_total<T>(args, d, launch_idx);
     if (blockIdx.x == 0) d->total_seen = total;
     S->chunk = chunk;
-    S->admitted = 1;
-    S->draining = 0;
     S->have_nxt = 0;
     S->long_vg = 0;
-    S->hint_live = 0xffffffffu;
-    S->hint_alive = 0;
-    if (kResolve) {
-      asm volatile("red.relaxed.gpu.global.max.u32 [%0], %1;" ::"l"(&d->ctl->cur), "r"(d->req_idx) : "memory");
-      S->admitted = admit(d) ? 1 : 0;
-      if (S->admitted) b = dequeue<true>(d, S);
-    }
     if (b < total) red_add_u32(&d->ctas_started, 1u);
     S->end = b < total ? min(b + chunk, total) : b;
     S->total = total;
@@ -396,6 +407,10 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     S->template set_cur<has_spread<T>::value>(0, b);
   }
   __syncthreads();
+  // thread 0: the prefetched queue word and live quota stay in registers
+  // across the body (a shared-memory store would wait for the atomic)
+  unsigned long long r_v = 0;
+  uint32_t r_live = 0;
   for (uint32_t k = 0;; k ^= 1u) {
     const SchedState::Cur c = S->cur[k];
     if (c.vg >= S->total) break;                 // RUN_TERMINATE
@@ -407,7 +422,8 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
         // for up to one VG duration.  So kernels whose VGs run long (where
         // that idle time dwarfs one queue round trip) dequeue just in time
         // once fewer than two waves of VGs remain
-        S->nxt = dequeue<kResolve>(d, S);
+        r_v = dequeue<kResolve>(d, S);
+        if (kResolve) r_live = d->governed ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
         S->have_nxt = 1;
       }
       S->t0 = globaltimer();
@@ -426,7 +442,18 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
       if (vg + 1 < S->end) {
         S->template set_cur<has_spread<T>::value>(k ^ 1u, vg + 1);
       } else {                                   // publish the prefetched chunk
-        const uint32_t nxt = S->have_nxt ? S->nxt : dequeue<kResolve>(d, S);   // tail: just in time
+        if (!S->have_nxt) {                      // tail: just in time
+          r_v = dequeue<kResolve>(d, S);
+          if (kResolve) r_live = d->governed ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
+        }
+        uint32_t nxt = kTerminate;
+        if (r_v != kEvicted) {
+          nxt = qa_next(r_v);
+          if (kResolve) {
+            S->hint_alive = qa_alive(r_v);   // admitted CTAs at our dequeue (incl. us)
+            S->hint_live = r_live;
+          }
+        }
         S->end = nxt < S->total ? min(nxt + S->chunk, S->total) : nxt;
         S->template set_cur<has_spread<T>::value>(k ^ 1u, nxt);
         S->have_nxt = 0;
@@ -471,7 +498,7 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
     if (threadIdx.x == 0) {
       if (dl->has_prev) wait_complete(dl - 1);  // launch l's inputs are complete
       atomicExch(&dl->topped, 1u);
-      __threadfence();
+      fence_acq_rel();
     }
     __syncthreads();
     const uint32_t cfg = dl->chunk | kCfgResolve | ((dl->flags & kFlagStamps) ? kCfgStamps : 0u);

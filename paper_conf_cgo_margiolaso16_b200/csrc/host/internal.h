@@ -24,6 +24,7 @@ struct InitParams {
   Desc* d;
   Ctl* ctl;               // RESOLVE control block, nullptr under STATIC
   uint32_t live_init;     // initial live quota of the main step
+  uint32_t main_step;     // the step the live quota governs
   uint32_t* coverage;     // nullptr unless verify
   accel_vg_record* trace; // nullptr unless ACCEL_REQ_TRACE
   uint32_t flags;

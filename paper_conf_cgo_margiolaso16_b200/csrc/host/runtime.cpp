@@ -120,12 +120,14 @@ struct DescHost {
   uint64_t ctl, coverage;
   uint32_t has_prev, pad_a;
   uint64_t trace;
-  uint32_t pad0[16];
+  uint32_t governed;
+  uint32_t pad0[15];
   // line 1
-  uint32_t next, pad1[31];
+  unsigned long long qa;  // alive << 32 | next
+  uint32_t pad1[30];
   // line 2
   unsigned long long t_first, t_last;
-  uint32_t total_seen, ctas_started, alive, max_alive, topped, admit_fail, evicted, last_live, adm, draining, pad2[18];
+  uint32_t total_seen, ctas_started, pad_alive, max_alive, topped, admit_fail, evicted, last_live, pad_adm, draining, pad2[18];
 };
 static_assert(sizeof(DescHost) == accel::kDescBytes, "host view of the descriptor");
 
@@ -260,7 +262,7 @@ int fetch_result(accel_ctx* ctx, Request* r) {
                          "[accel] coverage: req %llu tenant %d launch %u: %u bad VGs (first %u ran %u times), "
                          "total %u seen %u next %u topped %u alive %u refused %u evicted %u live %u\n",
                          (unsigned long long)r->id, r->tenant, s.first + l, bad, first_bad, got, s.total,
-                         d->total_seen, d->next, d->topped, d->alive, d->admit_fail, d->evicted, d->last_live);
+                         d->total_seen, (uint32_t)d->qa, d->topped, (uint32_t)(d->qa >> 32), d->admit_fail, d->evicted, d->last_live);
         }
       }
     r->cov_ok = ok ? 1 : 0;
@@ -284,6 +286,7 @@ int enqueue(accel_ctx* ctx, Request* r) {
   const bool resolve = shared && ctx->cfg.policy == ACCEL_POLICY_RESOLVE;
   p.ctl = resolve ? ctx->ctl_ptr(r->slot) : nullptr;
   p.live_init = r->steps[r->main_step].quota;
+  p.main_step = (uint32_t)r->main_step;
   p.coverage = r->cov;
   p.trace = r->trace;
   p.flags = kFlagStamps | (shared ? kFlagAlive : 0u);

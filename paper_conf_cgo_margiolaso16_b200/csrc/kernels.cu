@@ -46,12 +46,11 @@ __global__ void desc_init_kernel(const InitParams p, uint32_t n_desc) {
   d->ctl = p.ctl;
   d->coverage = p.coverage ? p.coverage + st.cov_offset + (size_t)r * st.total : nullptr;
   d->trace = p.trace ? p.trace + st.cov_offset + (size_t)r * st.total : nullptr;
+  d->governed = s == p.main_step ? 1u : 0u;
   d->t_first = ULLONG_MAX;
   d->t_last = 0;
   d->ctas_started = 0;
-  d->alive = 0;
   d->max_alive = 0;
-  d->adm = 0;
   d->admit_fail = 0;
   d->evicted = 0;
   d->draining = 0;
@@ -59,7 +58,7 @@ __global__ void desc_init_kernel(const InitParams p, uint32_t n_desc) {
   d->topped = 0;
   d->req_idx = i;
   d->has_prev = i > 0 ? 1u : 0u;
-  d->next = 0;
+  d->qa = 0;
 }
 
 __global__ void join_kernel(const Desc* last) {

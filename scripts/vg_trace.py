@@ -72,10 +72,12 @@ def main():
     ap.add_argument("tenant")
     ap.add_argument("size", nargs="?", default="default")
     ap.add_argument("--launch", type=int, default=-1, help="launch index to analyse (-1: the longest)")
+    ap.add_argument("--policy", default="static", choices=["static", "resolve"])
     a = ap.parse_args()
     d = synth.preset(a.tenant, a.size, seed=1)
     for mode in ("native", "persistent"):
-        acc = Accel(0, mode=abi.MODE_NATIVE if mode == "native" else abi.MODE_SHARED)
+        acc = Accel(0, mode=abi.MODE_NATIVE if mode == "native" else abi.MODE_SHARED,
+                    policy=abi.POLICY_RESOLVE if a.policy == "resolve" else abi.POLICY_STATIC)
         job = make_job(a.tenant, d)
         acc.run([job])                      # warm
         ids = acc.submit([job], trace=True)
@@ -91,6 +93,12 @@ def main():
         spans = [(tr[offs[i]:offs[i + 1]]["t_end_ns"].max() - tr[offs[i]:offs[i + 1]]["t_start_ns"][tr[offs[i]:offs[i + 1]]["t_start_ns"] > 0].min())
                  if (tr[offs[i]:offs[i + 1]]["t_start_ns"] > 0).any() else 0 for i in range(len(totals))]
         li = int(np.argmax(spans)) if a.launch < 0 else a.launch
+        if len(ls) > 1:
+            lsp = [(l.t_last_ns - l.t_first_ns) / 1e3 for l in ls]
+            gaps = [(ls[i + 1].t_first_ns - ls[i].t_last_ns) / 1e3 for i in range(len(ls) - 1)]
+            print(a.tenant, mode, "launches", len(ls), "span us mean %.1f" % np.mean(lsp),
+                  "gap us mean %.2f min %.2f" % (np.mean(gaps), np.min(gaps)),
+                  "request us %.1f" % ((ls[-1].t_last_ns - ls[0].t_first_ns) / 1e3), flush=True)
         part = tr[offs[li]:offs[li + 1]]
         print(a.tenant, mode, "launch", li, analyse(part, mode), flush=True)
         dur = (part["t_end_ns"].astype(np.int64) - part["t_start_ns"].astype(np.int64)) / 1e3
