@@ -407,6 +407,14 @@ def main():
                                                                       "frac": ach_iso / peak,
                                                                       "avg_launch_ms": avg_iso}}
     dom = max(roof, key=lambda t: tot[t]) if roof else None
+    # DRAM traffic per launch of the dominant kernel from the committed
+    # `ncu --set full` capture (scripts/ncu_traffic.py -> profiles/ncu_traffic.json)
+    tpath = os.path.join(ROOT, "profiles", "ncu_traffic.json")
+    if dom is not None and os.path.exists(tpath):
+        tr = json.load(open(tpath)).get(dom)
+        if tr:
+            roof[dom]["traffic"] = tr["dram_bytes_per_launch"]
+            roof[dom]["traffic_source"] = tr.get("source")
 
     launches_per_step = sum(1 + j.launches() for j in jobs)  # descriptor init + kernel launches
     h2d = sum(j.h2d_bytes() for j in jobs)
