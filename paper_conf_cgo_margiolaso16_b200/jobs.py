@@ -37,6 +37,14 @@ def _cdiv(a: int, b: int) -> int:
     return -(-a // b)
 
 
+# Roofline peaks for the non-HBM tenants: FP32 SIMT derived from
+# the guide's unit counts (148 SM x 128 FP32 lanes x 2 flop x 1.965 GHz); TF32
+# tensor = the measured bf16 dense peak (MEASURED_PEAKS.json, 1678.1 TF/s
+# burst) x the nominal TF32/BF16 ratio 1/2.
+FP32_SIMT_TFLOPS = 148 * 128 * 2 * 1.965e9 / 1e12
+TF32_TENSOR_TFLOPS = 1678.1 / 2
+
+
 @dataclass
 class Step:
     kernel: str
@@ -253,7 +261,7 @@ class CutcpJob(Job):
         # density (cutcp algorithmic work); ~15 flop each
         dens = self.d["natoms"] / self.d["box"] ** 3
         pairs = self.nx * self.ny * self.nz * dens * 4.0 / 3.0 * np.pi * self.d["cutoff"] ** 3
-        return {"pairs": pairs, "flops": 15.0 * pairs, "bound": "alu", "launches": 1}
+        return {"pairs": pairs, "flops": 15.0 * pairs, "bound": "alu", "launches": 1, "peak_tflops": FP32_SIMT_TFLOPS}
 
 
 class TpacfJob(Job):
@@ -281,7 +289,7 @@ class TpacfJob(Job):
     def work(self):
         n, S = self.n, self.S
         pairs = (1 + S) * n * (n - 1) // 2 + S * n * n
-        return {"pairs": pairs, "flops": 5.0 * pairs, "bound": "alu", "launches": 1}
+        return {"pairs": pairs, "flops": 5.0 * pairs, "bound": "alu", "launches": 1, "peak_tflops": FP32_SIMT_TFLOPS}
 
 
 class SpmvJob(Job):
@@ -322,7 +330,7 @@ class SgemmJob(Job):
 
     def work(self):
         f = 2.0 * self.m * self.n * self.k
-        return {"flops": f, "flops_per_launch": f, "bound": "alu", "launches": 1}
+        return {"flops": f, "flops_per_launch": f, "bound": "alu", "launches": 1, "peak_tflops": FP32_SIMT_TFLOPS}
 
 
 class SgemmTcJob(Job):
@@ -363,7 +371,7 @@ class SgemmTcJob(Job):
         f = 2.0 * self.m * self.n * self.k
         # roofline of the dominant (tc) launch: 3 tf32 products per algorithmic MAC
         return {"flops": f, "flops_per_launch": f, "bound": "tensor", "launches": 3, "skip_launches": 2,
-                "mma_flops": 3 * f}
+                "mma_flops": 3 * f, "peak_tflops": TF32_TENSOR_TFLOPS}
 
 
 class MriqJob(Job):
@@ -394,7 +402,7 @@ class MriqJob(Job):
     def work(self):
         pairs = self.numx * self.numk
         return {"pairs": pairs, "flops": 11.0 * pairs, "sfu": 2 * pairs, "bound": "alu", "launches": 2,
-                "skip_launches": 1, "flops_per_launch": 11.0 * pairs}
+                "skip_launches": 1, "flops_per_launch": 11.0 * pairs, "peak_tflops": FP32_SIMT_TFLOPS}
 
 
 JOBS = {"mop": MopJob, "stencil": StencilJob, "histo": HistoJob, "bfs": BfsJob, "cutcp": CutcpJob,

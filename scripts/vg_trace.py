@@ -109,6 +109,15 @@ def main():
         w1 = st0 < 5
         print("  first-wave VGs:", int(w1.sum()), "mean us", round(float(dur[w1].mean()), 0),
               "later mean us", round(float(dur[~w1].mean()), 0))
+        fw = part[w1]
+        fd = dur[w1]
+        ratios = []
+        for smv in np.unique(fw["sm"]):
+            dd = fd[fw["sm"] == smv]
+            if len(dd) > 1:
+                ratios.append(dd.max() / max(dd.min(), 1e-3))
+        print("  first wave, per SM max/min VG duration: median %.2f p90 %.2f" %
+              (float(np.median(ratios)), float(np.percentile(ratios, 90))))
         del ls
         torch.cuda.synchronize()
 
