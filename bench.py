@@ -239,7 +239,6 @@ def aggregate(allres: list[dict], world: int, steps: int, policy: str) -> dict:
     tmax = max(r["dev_ms"] for r in allres)
     emax = max(r["e2e_ms"] for r in allres)
     nmax = max(r["nat_ms"] for r in allres)
-    omax = max(r["oth_ms"] for r in allres)
     return {
         "tmax": tmax, "emax": emax, "nmax": nmax,
         "value": world * steps / (tmax / 1e3),
@@ -250,12 +249,13 @@ def aggregate(allres: list[dict], world: int, steps: int, policy: str) -> dict:
         "antt_sh": statistics.mean(u for r in allres for u in r["sh"]["ANTT"]),
         "antt_na": statistics.mean(u for r in allres for u in r["na"]["ANTT"]),
         "other": {
-            "policy": "static" if policy == "resolve" else "resolve",
-            "unfairness": gm([u for r in allres for u in r["ot"]["U"]]),
-            "stp": statistics.mean(u for r in allres for u in r["ot"]["STP"]),
-            "antt": statistics.mean(u for r in allres for u in r["ot"]["ANTT"]),
-            "mixes_per_s": world * steps / (omax / 1e3),
-            "throughput_speedup": nmax / omax,
+            name: {
+                "unfairness": gm([u for r in allres for u in r["ot"][name]["U"]]),
+                "stp": statistics.mean(u for r in allres for u in r["ot"][name]["STP"]),
+                "antt": statistics.mean(u for r in allres for u in r["ot"][name]["ANTT"]),
+                "mixes_per_s": world * steps / (max(r["oth_ms"][name] for r in allres) / 1e3),
+                "throughput_speedup": nmax / max(r["oth_ms"][name] for r in allres),
+            } for name in allres[0]["ot"]
         },
     }
 
@@ -269,8 +269,8 @@ def main():
     ap.add_argument("--config", default="c2", choices=["c1", "c2", "c5"])
     ap.add_argument("--impl", default="accel", choices=["accel", "reference"])
     ap.add_argument("--calib-reps", type=int, default=5)
-    ap.add_argument("--policy", default="resolve", choices=["resolve", "static"],
-                    help="SHARED-mode policy of the timed (headline) run; the other is reported too")
+    ap.add_argument("--policy", default="fair", choices=["fair", "resolve", "static", "partition"],
+                    help="SHARED-mode policy of the timed (headline) run; the others are reported too")
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--out", default=None, help="also write the JSON line here")
     args = ap.parse_args()
@@ -300,9 +300,11 @@ def main():
         flush_buf.fill_(1.0)
         torch.cuda.synchronize()
 
-    POL = {"resolve": abi.POLICY_RESOLVE, "static": abi.POLICY_STATIC}
+    POL = {"fair": abi.POLICY_FAIR, "resolve": abi.POLICY_RESOLVE, "static": abi.POLICY_STATIC,
+           "partition": abi.POLICY_PARTITION}
+    hints = {}   # FAIR: isolated-time profile per tenant (from the calibration below)
     head_pol = POL[args.policy]
-    other_pol = POL["static" if args.policy == "resolve" else "resolve"]
+    other_pols = [p for p in POL if p != args.policy]
 
     def run_group(js, mode, e2e=False, launch_events=False, policy=None):
         policy = head_pol if policy is None else policy
@@ -310,7 +312,8 @@ def main():
             acc.set_mode(mode, policy)
         flush()
         acc.epoch()
-        ids = acc.submit(js, e2e=e2e, launch_events=launch_events)
+        iso = [hints.get(j.name, 0.0) for j in js] if policy == abi.POLICY_FAIR else None
+        ids = acc.submit(js, e2e=e2e, launch_events=launch_events, isolated_ms=iso)
         acc.sync()
         st = [acc.stats(i) for i in ids]
         lt = [acc.launch_times(i, j.launches()) for i, j in zip(ids, js)] if launch_events else None
@@ -319,8 +322,8 @@ def main():
 
     # -- correctness pass (untimed): coverage of every VG, both modes
     with Accel(device=local, mode=abi.MODE_SHARED, verify=True) as vacc:
-        for mode in (abi.MODE_NATIVE, abi.MODE_SHARED):
-            vacc.set_mode(mode)
+        for mode, pol in [(abi.MODE_NATIVE, abi.POLICY_STATIC)] + [(abi.MODE_SHARED, POL[p]) for p in POL]:
+            vacc.set_mode(mode, pol)
             st = vacc.run(jobs)
             assert all(s.coverage_ok == 1 for s in st), "coverage check failed"
 
@@ -337,6 +340,7 @@ def main():
             if mode == abi.MODE_SHARED:
                 iso_launch[j.name] = lts
     ta = [iso_native[t] for t in tenants]
+    hints.update(iso_native)
 
     def steps_loop(mode, k, e2e=False, policy=None):
         out = []
@@ -356,8 +360,10 @@ def main():
         dist.barrier()
     steps_loop(abi.MODE_NATIVE, args.warmup)
     native = steps_loop(abi.MODE_NATIVE, args.steps)
-    steps_loop(abi.MODE_SHARED, 1, policy=other_pol)
-    other = steps_loop(abi.MODE_SHARED, args.steps, policy=other_pol)
+    other = {}
+    for p in other_pols:
+        steps_loop(abi.MODE_SHARED, 1, policy=POL[p])
+        other[p] = steps_loop(abi.MODE_SHARED, args.steps, policy=POL[p])
     steps_loop(abi.MODE_SHARED, 1, e2e=True)
     e2e = steps_loop(abi.MODE_SHARED, args.steps, e2e=True)
 
@@ -375,7 +381,8 @@ def main():
         return {"makespan_ms": mk, "U": U, "STP": STP, "ANTT": ANTT, "O": OV,
                 "ts_ms": [[s.elapsed_ms for s in st] for st, _ in runs]}
 
-    sh, na, ee, ot = summarize(shared), summarize(native), summarize(e2e), summarize(other)
+    sh, na, ee = summarize(shared), summarize(native), summarize(e2e)
+    ot = {p: summarize(v) for p, v in other.items()}
     dev_ms = sum(sh["makespan_ms"])
     e2e_ms = sum(ee["makespan_ms"])
     nat_ms = sum(na["makespan_ms"])
@@ -416,12 +423,13 @@ def main():
             roof[dom]["traffic"] = tr["dram_bytes_per_launch"]
             roof[dom]["traffic_source"] = tr.get("source")
 
-    launches_per_step = sum(1 + j.launches() for j in jobs)  # descriptor init + kernel launches
+    # descriptor init + kernel launches (PARTITION: one grid per step + the join kernel)
+    launches_per_step = sum((2 + len(j.steps)) if args.policy == "partition" else (1 + j.launches()) for j in jobs)
     h2d = sum(j.h2d_bytes() for j in jobs)
     d2h = sum(j.d2h_bytes() for j in jobs)
 
     local_res = {"rank": rank, "dev_ms": dev_ms, "e2e_ms": e2e_ms, "nat_ms": nat_ms,
-                 "oth_ms": sum(ot["makespan_ms"]), "tenants": tenants, "sh": sh, "na": na, "ot": ot,
+                 "oth_ms": {p: sum(v["makespan_ms"]) for p, v in ot.items()}, "tenants": tenants, "sh": sh, "na": na, "ot": ot,
                  "quotas": [[s.quota_initial, s.quota_min, s.quota_max, s.resolves] for s in shared[-1][0]],
                  "clk": clk.summary()}
     if world > 1:
@@ -444,7 +452,8 @@ def main():
         tmax, emax, nmax, value = agg["tmax"], agg["emax"], agg["nmax"], agg["value"]
         U_sh, U_na, stp_sh, stp_na = agg["U_sh"], agg["U_na"], agg["stp_sh"], agg["stp_na"]
         antt_sh, antt_na, other_sum = agg["antt_sh"], agg["antt_na"], agg["other"]
-        other_sum["T_s_ms"] = dict(zip(tenants, np.mean(allres[0]["ot"]["ts_ms"], 0).tolist()))
+        for p in other_sum:
+            other_sum[p]["T_s_ms"] = dict(zip(tenants, np.mean(allres[0]["ot"][p]["ts_ms"], 0).tolist()))
         clocks = allres[0]["clk"]
         line = {
             "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": args.steps,
@@ -469,7 +478,7 @@ def main():
                 "dispatch_overhead": {t: iso_persist[t] / iso_native[t] - 1 for t in tenants},
                 "native_mixes_per_s": world * args.steps / (nmax / 1e3),
                 "quotas_last_step": dict(zip(tenants, allres[0]["quotas"])),
-                "other_policy": other_sum,
+                "other_policies": other_sum,
             },
             "e2e": {"value": world * args.steps / (emax / 1e3), "unit": UNIT,
                     "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h},

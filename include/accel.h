@@ -50,8 +50,26 @@ typedef enum { ACCEL_MODE_NATIVE = 0, ACCEL_MODE_SHARED = 1 } accel_mode;
 /* STATIC: a quota is fixed at launch (§2.5, "bound to
  * the resources initially allocated").  RESOLVE: quotas are recomputed on every
  * arrival and departure (BASELINE.json north star): shrinking lowers a live
- * quota word read at each dequeue, growing launches extra CTAs. */
-typedef enum { ACCEL_POLICY_STATIC = 0, ACCEL_POLICY_RESOLVE = 1 } accel_policy;
+ * quota word read at each dequeue, growing launches extra CTAs.
+ * PARTITION: whole SMs are the unit of sharing (the CU split of PAPER.md
+ * Fig. 3b): accel_solve_sms gives each active request s_i SMs;
+ * its persistent CTAs claim SMs on the device (a per-SM owner word) and run
+ * c_i per SM, padded in shared memory so that no other kernel's CTA fits
+ * beside them; re-solved on every arrival and departure (an SM is handed over
+ * at a VG boundary).  One persistent grid serves all launches of a step. */
+/* FAIR: RESOLVE whose weights follow the requests' measured slowdowns: the
+ * monitor reads each running request's completed VGs every few hundred
+ * microseconds, estimates its slowdown so far against its isolated time
+ * (accel_request.isolated_ns, a profile the caller supplies) and re-solves
+ * with weights growing with the slowdown, so laggards get a larger share
+ * (§2.2, "changing the sharing ratio"; DESIGN.md
+ * R-fair-1..3).  Requests without a hint keep the neutral weight. */
+typedef enum {
+  ACCEL_POLICY_STATIC = 0,
+  ACCEL_POLICY_RESOLVE = 1,
+  ACCEL_POLICY_PARTITION = 2,
+  ACCEL_POLICY_FAIR = 3
+} accel_policy;
 
 #define ACCEL_ALL UINT64_MAX
 #define ACCEL_MAX_TENANTS 16
@@ -104,6 +122,8 @@ typedef struct {
   int32_t regs;               /* regs/thread for the solver; 0 = query attrs   */
   uint32_t chunk;             /* VGs per dequeue (§6.4); 0 = default  */
   uint32_t args_size;         /* sizeof the kernel's argument struct           */
+  const void *partition_fn;   /* host stub of accel_topup<T, PARTITION>; NULL =
+                                 the kernel cannot run under ACCEL_POLICY_PARTITION */
 } accel_kernel_desc;
 
 /* Fill *out with a built-in tenant kernel: "mop", "stencil", "histo", "bfs",
@@ -126,6 +146,8 @@ typedef struct {
   int32_t static_smem;            /* static shared memory of the instance      */
   int32_t occ_persistent;         /* cudaOccupancyMaxActiveBlocksPerMultiprocessor */
   int32_t occ_native;
+  int32_t occ_partition;          /* PARTITION: CTAs per SM c_i (0: none)       */
+  uint32_t partition_smem;        /* PARTITION: padded dynamic smem per CTA     */
 } accel_kernel_info;
 int accel_kernel_info_get(accel_ctx *ctx, int32_t kernel_id, accel_kernel_info *out);
 
@@ -143,6 +165,12 @@ typedef struct {
   const void *args;      /* points to the kernel's argument struct (copied)      */
   uint32_t args_size;    /* must equal the registered args_size                  */
   uint32_t repeat;       /* launches of this step, >= 1                          */
+  const uint32_t *order_device; /* dequeue order (SHARED mode): the t-th VG handed out
+                           is order_device[t], a permutation of 0..G-1 in device
+                           memory, caller-owned (e.g. most expensive VGs first, so
+                           that the cheapest ones form the tail); NULL = increasing
+                           linear order.  Static-grid kernels only.  NATIVE mode
+                           ignores it (hardware order).                            */
 } accel_launch;
 
 typedef struct { void *dst_device; int32_t value; uint64_t bytes; } accel_clear;
@@ -171,6 +199,11 @@ typedef struct {
   const accel_copy *h2d;
   uint32_t n_d2h;             /* device->host copies after the last launch      */
   const accel_copy *d2h;
+  uint64_t isolated_ns;       /* ACCEL_POLICY_FAIR: the request's isolated run
+                                 time (a profile); 0 = unknown (neutral weight) */
+  uint64_t vgs_hint;          /* FAIR: VGs the request will run; 0 = the sum of
+                                 its static grids (dynamic-total kernels such as
+                                 bfs run fewer: pass 0 AND isolated_ns = 0)     */
 } accel_request;
 
 /* Submit one request (solver run over the active set incl. this one).
@@ -246,6 +279,18 @@ int accel_demand_of(const accel_caps *caps, uint32_t block_threads, uint32_t reg
 /* The share solver of PAPER.md §3 (closed form + per-SM feasibility + greedy),
  * k requests in arrival order -> quota_out[k]. */
 int accel_solve(const accel_caps *caps, const accel_demand *d, int32_t k, uint32_t *quota_out);
+/* SM-granular variant (ACCEL_POLICY_PARTITION; DESIGN.md R-part-1..4): the
+ * same closed form + class-symmetric greedy with whole SMs as the one device
+ * total.  sms_out[k] = SMs per request (sum <= caps->sms, each <= ceil(G/c));
+ * ctas_per_sm_out[k] (may be NULL) = c_i, CTAs of the kernel alone on one SM.
+ * ACCEL_ENOFIT if a CTA fits no SM. */
+int accel_solve_sms(const accel_caps *caps, const accel_demand *d, int32_t k, uint32_t *sms_out,
+                    uint32_t *ctas_per_sm_out);
+/* ACCEL_POLICY_FAIR weights (DESIGN.md R-fair-2): from the slowdowns so far
+ * slowdown[k] (> 0; <= 0 = not yet known -> the neutral weight 16),
+ * weight_out[i] = round(16 * (slowdown_i / g)^2) clamped to [1, 1024], g the
+ * geometric mean of the known slowdowns. */
+int accel_fair_weights(const double *slowdown, int32_t k, uint32_t *weight_out);
 
 typedef struct {
   double unfairness;  /* max IS / min IS */

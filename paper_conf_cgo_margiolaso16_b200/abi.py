@@ -23,7 +23,7 @@ ACCEL_ENOTREADY = -7
 ERRORS = {0: "ACCEL_OK", -1: "ACCEL_EINVAL", -2: "ACCEL_ENOFIT", -3: "ACCEL_ECUDA",
           -4: "ACCEL_ESTATE", -5: "ACCEL_ECOVERAGE", -6: "ACCEL_ENOMEM", -7: "ACCEL_ENOTREADY"}
 MODE_NATIVE, MODE_SHARED = 0, 1
-POLICY_STATIC, POLICY_RESOLVE = 0, 1
+POLICY_STATIC, POLICY_RESOLVE, POLICY_PARTITION, POLICY_FAIR = 0, 1, 2, 3
 ACCEL_ALL = 2**64 - 1
 MAX_TENANTS = 16
 MAX_STEPS = 8
@@ -50,16 +50,19 @@ class accel_kernel_desc(C.Structure):
     _fields_ = [("name", C.c_char_p), ("persistent_fn", vp), ("persistent_resolve_fn", vp), ("native_fn", vp),
                 ("topup_fn", vp),
                 ("block", accel_dim3),
-                ("dyn_smem", u32), ("regs", i32), ("chunk", u32), ("args_size", u32)]
+                ("dyn_smem", u32), ("regs", i32), ("chunk", u32), ("args_size", u32),
+                ("partition_fn", vp)]
 
 
 class accel_kernel_info(C.Structure):
     _fields_ = [("thr", u32), ("regs", u32), ("smem", u32), ("cta", u32), ("num_regs", i32),
-                ("static_smem", i32), ("occ_persistent", i32), ("occ_native", i32)]
+                ("static_smem", i32), ("occ_persistent", i32), ("occ_native", i32),
+                ("occ_partition", i32), ("partition_smem", u32)]
 
 
 class accel_launch(C.Structure):
-    _fields_ = [("kernel_id", i32), ("grid", accel_dim3), ("args", vp), ("args_size", u32), ("repeat", u32)]
+    _fields_ = [("kernel_id", i32), ("grid", accel_dim3), ("args", vp), ("args_size", u32), ("repeat", u32),
+                ("order_device", vp)]
 
 
 class accel_clear(C.Structure):
@@ -73,7 +76,8 @@ class accel_copy(C.Structure):
 class accel_request(C.Structure):
     _fields_ = [("tenant", i32), ("flags", u32), ("weight", u32), ("main_step", i32), ("n_steps", u32), ("steps", C.POINTER(accel_launch)),
                 ("n_clear", u32), ("clear", C.POINTER(accel_clear)), ("n_h2d", u32),
-                ("h2d", C.POINTER(accel_copy)), ("n_d2h", u32), ("d2h", C.POINTER(accel_copy))]
+                ("h2d", C.POINTER(accel_copy)), ("n_d2h", u32), ("d2h", C.POINTER(accel_copy)),
+                ("isolated_ns", u64), ("vgs_hint", u64)]
 
 
 class accel_req_stats(C.Structure):
@@ -159,7 +163,7 @@ EXPORTS = [
     "accel_init", "accel_finalize", "accel_set_mode", "accel_last_error", "accel_builtin_kernel",
     "accel_builtin_count", "accel_builtin_name", "accel_kernel_register", "accel_kernel_info_get",
     "accel_submit", "accel_submit_group", "accel_sync", "accel_epoch", "accel_stats", "accel_release",
-    "accel_tenant_stream", "accel_launch_times", "accel_launch_stats", "accel_vg_trace", "accel_demand_of", "accel_solve", "accel_metrics", "accel_overlap", "accel_tma_map_2d",
+    "accel_tenant_stream", "accel_launch_times", "accel_launch_stats", "accel_vg_trace", "accel_demand_of", "accel_solve", "accel_solve_sms", "accel_fair_weights", "accel_metrics", "accel_overlap", "accel_tma_map_2d",
 ]
 
 
@@ -197,6 +201,8 @@ def _load() -> C.CDLL:
         "accel_vg_trace": (i32, [vp, u64, P(accel_vg_record), u64, P(u64)]),
         "accel_demand_of": (i32, [P(accel_caps), u32, u32, u32, u32, u32, P(accel_demand)]),
         "accel_solve": (i32, [P(accel_caps), P(accel_demand), i32, P(u32)]),
+        "accel_solve_sms": (i32, [P(accel_caps), P(accel_demand), i32, P(u32), P(u32)]),
+        "accel_fair_weights": (i32, [P(f64), i32, P(u32)]),
         "accel_metrics": (i32, [P(f64), P(f64), i32, P(accel_mix_metrics)]),
         "accel_overlap": (i32, [P(f64), P(f64), i32, P(f64)]),
         "accel_tma_map_2d": (i32, [vp, vp, u64, u64, u64, u32, u32, i32]),
@@ -330,6 +336,23 @@ def accel_solve(demands: list[accel_demand], caps: accel_caps | None = None) -> 
     arr = (accel_demand * max(k, 1))(*demands)
     out = (u32 * max(k, 1))()
     check(lib.accel_solve(C.byref(caps or accel_caps()), arr, k, out))
+    return list(out)[:k]
+
+
+def accel_solve_sms(demands: list[accel_demand], caps: accel_caps | None = None) -> tuple[list[int], list[int]]:
+    """SM-granular partition: (SMs per request, CTAs per SM per request)."""
+    k = len(demands)
+    arr = (accel_demand * max(k, 1))(*demands)
+    sms = (u32 * max(k, 1))()
+    per = (u32 * max(k, 1))()
+    check(lib.accel_solve_sms(C.byref(caps or accel_caps()), arr, k, sms, per))
+    return list(sms)[:k], list(per)[:k]
+
+
+def accel_fair_weights(slowdowns: list[float]) -> list[int]:
+    k = len(slowdowns)
+    out = (u32 * max(k, 1))()
+    check(lib.accel_fair_weights((f64 * max(k, 1))(*slowdowns), k, out))
     return list(out)[:k]
 
 

@@ -20,7 +20,9 @@
 // The body never reads blockIdx/gridDim (the `mop` test catches that), keeps
 // no state across VGs and never waits on another CTA.
 //   accel_persistent<T>: the reduced-grid scheduling kernel (Fig. 8b dyn_sched).
-//   accel_topup<T>:      RESOLVE growth grids (sticky across a step's launches).
+//   accel_topup<T, P>:   sticky grids that follow a step's launches: RESOLVE
+//                        growth grids (P = false); under PARTITION (P = true)
+//                        every grid of a request (SM claims, see part_claim).
 //   accel_native<T>:     the same body on the original grid (Fig. 1a baseline).
 //
 // RESOLVE policy (BASELINE.json north star; not in the paper, whose kernels
@@ -47,9 +49,12 @@ namespace accel {
 
 // Per-request control block (device memory).
 struct Ctl {
-  uint32_t live;   // live quota (RESOLVE)
-  uint32_t cur;    // highest request-relative launch index started
-  uint32_t pad[2];
+  uint32_t live;      // live quota (RESOLVE)
+  uint32_t cur;       // highest request-relative launch index started
+  uint32_t sm_quota;  // PARTITION: SMs the request may own (host-written)
+  uint32_t sm_count;  // PARTITION: SMs it owns (claims - releases)
+  uint32_t done_vgs;  // FAIR: VGs completed by the request (progress, read by the host monitor)
+  uint32_t pad[3];
 };
 
 // Virtual NDRange of ONE launch ("Virtual Kernel Execution
@@ -75,7 +80,12 @@ struct alignas(128) Desc {
   uint32_t governed;       // RESOLVE: this launch belongs to the request's main
                            // step, whose CTA count the live quota governs (the
                            // other steps keep their own solved grid)
-  uint32_t pad0[15];
+  uint32_t tok;            // PARTITION: owner token of the request (slot + 1)
+  uint32_t* owner;         // PARTITION: per-SM owner words of the context
+  uint32_t last_step;      // PARTITION: launch of the request's last step
+  uint32_t ctas_per_sm;    // PARTITION: c_i of the step's kernel
+  const uint32_t* order;   // dequeue order (ticket t -> VG order[t]), nullptr = linear
+  uint32_t pad0[8];
   // ---- line 1: the software queue head (RUN_TERMINATE when >= total) in the
   // low 32 bits, the admitted CTA count (`alive`, RESOLVE) in the high 32
   unsigned long long qa;
@@ -108,7 +118,7 @@ __device__ __forceinline__ void red_add_u32(uint32_t* p, uint32_t v) {
   asm volatile("red.relaxed.gpu.global.add.u32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
 }
 
-enum : uint32_t { kFlagStamps = 1u, kFlagAlive = 2u };
+enum : uint32_t { kFlagStamps = 1u, kFlagAlive = 2u, kFlagProgress = 4u };
 
 // Desc::qa = alive << 32 | next
 constexpr unsigned long long kAlive1 = 1ull << 32;
@@ -282,6 +292,8 @@ struct SchedState {
   uint32_t nxt;        // prefetched chunk (valid if have_nxt)
   uint32_t* coverage;
   accel_vg_record* trace;
+  const uint32_t* order;   // dequeue order of the launch (nullptr: linear / spread)
+  uint32_t* progress;      // FAIR: Ctl::done_vgs (nullptr: not tracked)
   unsigned long long t0;   // trace: start of the current VG
   // RESOLVE, thread 0: view of the live quota and the admitted count, loaded
   // right after each dequeue and used at the next one, so the check adds no
@@ -290,18 +302,87 @@ struct SchedState {
   uint8_t have_nxt, admitted, draining;
   uint8_t over;        // RESOLVE: admitted over the live quota -> leave at the next dequeue
   uint8_t long_vg;     // the last VG ran longer than kLongVgNs
+  uint8_t left;        // PARTITION: the CTA gave up its SM (leaves the sticky loop)
+  // PARTITION, thread 0: this CTA's SM, the request's token, the owner words,
+  // and the views loaded right after the last dequeue (used at the next)
+  uint32_t sm, tok;
+  uint32_t* owner;
+  uint32_t hint_owner, hint_q, hint_c;
   template <bool kSpread>
   __device__ __forceinline__ void set_cur(uint32_t k, uint32_t vg) {
     cur[k].vg = vg;
     if (vg < total) {
       uint32_t id = vg;
-      if constexpr (kSpread) id = (uint32_t)(((uint64_t)vg * spread) % total);
+      if (order != nullptr) {
+        id = __ldg(order + vg);
+      } else if constexpr (kSpread) {
+        id = (uint32_t)(((uint64_t)vg * spread) % total);
+      }
       cur[k].id = id;
       const VirtualBlock b = decode(id, gx, gy, gz, launch_idx);
       cur[k].x = b.x; cur[k].y = b.y; cur[k].z = b.z;
     }
   }
 };
+
+// ---------------------------------------------------------------------------
+// PARTITION policy (DESIGN.md R-part-*): whole SMs per request.  owner[sm] is
+// 0 (free), tok (owned), tok | kOwnRel (being handed over: claimable by any
+// request under its SM quota, including tok itself) or tok | kOwnClaim (a CTA
+// of tok is claiming it right now).  A request's CTAs are padded in shared
+// memory so that c_i of them fill an SM: no other kernel's CTA fits beside
+// them, which is what makes the partition hold on the hardware.
+constexpr uint32_t kOwnRel = 0x80000000u;
+constexpr uint32_t kOwnClaim = 0x40000000u;
+
+__device__ __forceinline__ unsigned long long ld_relaxed_u64(const void* p) {
+  unsigned long long v;
+  asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+  return v;
+}
+
+// Thread 0 at CTA start: make this SM the request's (or find it already is).
+// One CTA per SM claims (the kOwnClaim state); the claim takes a ticket on the
+// request's SM count, so at most sm_quota SMs are ever owned.
+__device__ __forceinline__ bool part_claim(uint32_t* owner, Ctl* ctl, uint32_t sm, uint32_t tok) {
+  for (;;) {
+    const uint32_t o = ld_volatile(&owner[sm]);
+    if (o == tok) return true;
+    if (o == (tok | kOwnClaim)) {  // a sibling CTA is claiming this SM
+      __nanosleep(64);
+      continue;
+    }
+    if (o != 0 && !(o & kOwnRel)) return false;  // another request's SM
+    if (atomicCAS(&owner[sm], o, tok | kOwnClaim) != o) continue;
+    const uint32_t cnt = atomicAdd(&ctl->sm_count, 1u);
+    if (cnt < ld_volatile(&ctl->sm_quota)) {
+      atomicExch(&owner[sm], tok);
+      return true;
+    }
+    atomicSub(&ctl->sm_count, 1u);
+    atomicExch(&owner[sm], o);  // at quota: give it back as it was
+    return false;
+  }
+}
+
+// Thread 0 at a dequeue: must this CTA leave its SM?  o_h, q_h, c_h are the
+// owner word and the request's (quota, count) as loaded after the previous
+// dequeue.  Leaves if the SM is no longer the request's; if the request owns
+// more SMs than its quota, the first CTA of an SM to get here marks the SM as
+// handed over (its siblings see the mark at their next dequeue) -- one ticket
+// on the count per SM, so exactly count - quota SMs are released.
+__device__ __forceinline__ bool part_leave(uint32_t* owner, Ctl* ctl, uint32_t sm, uint32_t tok,
+                                           uint32_t o_h, uint32_t q_h, uint32_t c_h) {
+  if (o_h != tok) return true;
+  if (c_h <= q_h) return false;
+  if (atomicCAS(&owner[sm], tok, tok | kOwnRel) != tok) return true;  // a sibling released it
+  const uint32_t cnt = atomicSub(&ctl->sm_count, 1u);
+  if (cnt > ld_volatile(&ctl->sm_quota)) return true;
+  atomicAdd(&ctl->sm_count, 1u);  // enough SMs were released meanwhile: keep it
+  if (atomicCAS(&owner[sm], tok | kOwnRel, tok) == (tok | kOwnRel)) return false;
+  atomicSub(&ctl->sm_count, 1u);  // claimed by another request in between
+  return true;
+}
 
 // One dequeue (Fig. 8b line 26, rt_sched_wgroup): one 64-bit
 // atomicAdd of `chunk` on the queue word, which also returns the admitted
@@ -313,13 +394,16 @@ struct SchedState {
 // until retire(), after that VG's results are written.  Returns the raw queue
 // word (kEvicted when the CTA left).
 constexpr unsigned long long kEvicted = ~0ull;
-template <bool kResolve>
+template <bool kResolve, bool kPart = false>
 __device__ __forceinline__ unsigned long long dequeue(Desc* d, SchedState* S) {
-  if (kResolve && (S->over || S->hint_alive > S->hint_live)) {
+  const bool part_out =
+      kPart && part_leave(S->owner, d->ctl, S->sm, S->tok, S->hint_owner, S->hint_q, S->hint_c);
+  if (kResolve && (part_out || S->over || S->hint_alive > S->hint_live)) {
     atomicAdd(&d->draining, 1u);
     fence_acq_rel();   // draining visible before alive drops
     bool left = false;
-    if (S->over) {
+    if (S->over || part_out) {
+      if (part_out) S->left = 1;
       atomicAdd(&d->qa, kAliveNeg);
       left = true;
     } else {
@@ -358,7 +442,7 @@ __device__ __forceinline__ void retire(Desc* d, uint32_t cfg, const SchedState* 
 constexpr unsigned long long kLongVgNs = 40000;   // 40 us: ~20 queue round trips
 
 // Serve one launch: admission, dequeue loop, retire.  All threads call it.
-template <class T, bool kResolve>
+template <class T, bool kResolve, bool kPart = false>
 __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, char* smem,
                                       SchedState* S, uint32_t cfg, uint32_t cta_tag) {
   if (threadIdx.x == 0) {    // master work-item: environment init (rt_env_init)
@@ -369,6 +453,11 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     S->over = 0;
     if (!kResolve) {
       b = qa_next(atomicAdd(&d->qa, (unsigned long long)chunk));   // issued before anything else
+    } else if (kPart && part_leave(S->owner, d->ctl, S->sm, S->tok, S->hint_owner, S->hint_q, S->hint_c)) {
+      // PARTITION: the SM was handed over between two launches: leave unadmitted
+      S->left = 1;
+      S->admitted = 0;
+      b = kTerminate;
     } else {
       // admission and first dequeue in one atomic; an arrival over the live
       // quota runs the chunk it got and leaves at its next dequeue
@@ -389,7 +478,8 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     if (cfg & kCfgStamps) red_min_u64(&d->t_first, globaltimer());
     const uint32_t launch_idx = d->launch_idx;
     const uint32_t total = vg_total<T>(args, d, launch_idx);
-    if (blockIdx.x == 0) d->total_seen = total;
+    // (PARTITION: any CTA may be the only one that reaches this launch)
+    if (kPart ? ld_volatile(&d->total_seen) == kTerminate : blockIdx.x == 0) d->total_seen = total;
     S->chunk = chunk;
     S->have_nxt = 0;
     S->long_vg = 0;
@@ -402,15 +492,17 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     S->launch_idx = launch_idx;
     S->coverage = d->coverage;
     S->trace = d->trace;
+    S->order = d->order;
+    S->progress = (d->flags & kFlagProgress) ? &d->ctl->done_vgs : nullptr;
     S->spread = has_spread<T>::value ? spread_factor(total) : 0u;
-    S->prefetch_window = 2u * chunk * gridDim.x;
+    S->prefetch_window = 2u * chunk * (kPart ? d->ctas_per_sm * S->hint_q : gridDim.x);
     S->template set_cur<has_spread<T>::value>(0, b);
   }
   __syncthreads();
   // thread 0: the prefetched queue word and live quota stay in registers
   // across the body (a shared-memory store would wait for the atomic)
-  unsigned long long r_v = 0;
-  uint32_t r_live = 0;
+  unsigned long long r_v = 0, r_qc = 0;
+  uint32_t r_live = 0, r_own = 0;
   for (uint32_t k = 0;; k ^= 1u) {
     const SchedState::Cur c = S->cur[k];
     if (c.vg >= S->total) break;                 // RUN_TERMINATE
@@ -422,8 +514,12 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
         // for up to one VG duration.  So kernels whose VGs run long (where
         // that idle time dwarfs one queue round trip) dequeue just in time
         // once fewer than two waves of VGs remain
-        r_v = dequeue<kResolve>(d, S);
+        r_v = dequeue<kResolve, kPart>(d, S);
         if (kResolve) r_live = d->governed ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
+        if (kPart) {
+          r_own = ld_relaxed(&S->owner[S->sm]);
+          r_qc = ld_relaxed_u64(&d->ctl->sm_quota);
+        }
         S->have_nxt = 1;
       }
       S->t0 = globaltimer();
@@ -437,14 +533,24 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     if (threadIdx.x == 0) {
       const uint32_t vg = S->cur[k].vg, id = S->cur[k].id;
       if (S->coverage != nullptr) atomicAdd(&S->coverage[id], 1u);
+      if (S->progress != nullptr) red_add_u32(S->progress, 1u);
       if (S->trace != nullptr) trace_vg(S->trace, id, S->t0, cta_tag);
       S->long_vg = globaltimer() - S->t0 > kLongVgNs;
       if (vg + 1 < S->end) {
         S->template set_cur<has_spread<T>::value>(k ^ 1u, vg + 1);
       } else {                                   // publish the prefetched chunk
         if (!S->have_nxt) {                      // tail: just in time
-          r_v = dequeue<kResolve>(d, S);
+          r_v = dequeue<kResolve, kPart>(d, S);
           if (kResolve) r_live = d->governed ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
+          if (kPart) {
+            r_own = ld_relaxed(&S->owner[S->sm]);
+            r_qc = ld_relaxed_u64(&d->ctl->sm_quota);
+          }
+        }
+        if (kPart) {
+          S->hint_owner = r_own;
+          S->hint_q = (uint32_t)r_qc;
+          S->hint_c = (uint32_t)(r_qc >> 32);
         }
         uint32_t nxt = kTerminate;
         if (r_v != kEvicted) {
@@ -482,29 +588,62 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
 // RESOLVE top-up grid: d = first launch of the request step, `sticky` =
 // launches in the step; starts at the request's current launch and follows
 // the step's later launches (each only once its predecessor completed).
-template <class T>
+// PARTITION (kPart): the same loop is the request's ONLY kind of grid -- the
+// main grid of every step (c_i x S CTAs on the tenant stream) and the growth
+// grids -- and each CTA first claims its SM (part_claim); a CTA whose SM is
+// not the request's leaves at once, unless the request owns no SM at all
+// (then it serves one chunk as a guest, so a request can never starve).
+template <class T, bool kPart>
 __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
     accel_topup(const typename T::Args args, Desc* __restrict__ d, uint32_t sticky) {
   extern __shared__ __align__(128) char smem[];
   __shared__ SchedState S;
-  __shared__ uint32_t s_l;
+  __shared__ uint32_t s_l, s_ok;
   if (threadIdx.x == 0) {
     const uint32_t cur = ld_volatile(&d->ctl->cur);
     s_l = cur > d->req_idx ? cur - d->req_idx : 0u;
+    s_ok = 1;
+    S.left = 0;
+    if (kPart) {
+      S.sm = smid();
+      S.tok = d->tok;
+      S.owner = d->owner;
+      const Desc* last = d + (sticky - 1);
+      const uint32_t lt = ld_volatile(&last->total_seen);
+      const bool finished = s_l >= sticky || (lt != kTerminate && qa_next(ld_volatile_u64(&last->qa)) >= lt);
+      bool ok = !finished && part_claim(S.owner, d->ctl, S.sm, S.tok);
+      const unsigned long long qc = ld_relaxed_u64(&d->ctl->sm_quota);
+      S.hint_q = (uint32_t)qc;
+      S.hint_c = (uint32_t)(qc >> 32);
+      // guest: the request owns no SM (all of them are owned by others): run
+      // one chunk here (admitted on a pretended owner view) and leave at the
+      // next dequeue, whose fresh view shows the real owner
+      s_ok = ok || (!finished && S.hint_c == 0);
+      S.hint_owner = s_ok ? S.tok : 0u;
+    }
   }
   __syncthreads();
+  if (!s_ok) return;
   for (uint32_t l = s_l; l < sticky; ++l) {
     Desc* dl = d + l;
     if (threadIdx.x == 0) {
       if (dl->has_prev) wait_complete(dl - 1);  // launch l's inputs are complete
-      atomicExch(&dl->topped, 1u);
-      fence_acq_rel();
+      if (!kPart) {
+        atomicExch(&dl->topped, 1u);
+        fence_acq_rel();
+      }
     }
     __syncthreads();
     const uint32_t cfg = dl->chunk | kCfgResolve | ((dl->flags & kFlagStamps) ? kCfgStamps : 0u);
-    serve<T, true>(args, dl, smem, &S, cfg, blockIdx.x | 0x80000000u);
+    serve<T, true, kPart>(args, dl, smem, &S, cfg, blockIdx.x | (kPart ? 0u : 0x80000000u));
     __syncthreads();
+    if (kPart && S.left) return;
   }
+  // the step's last launch is exhausted: free the SM (one CTA per SM wins the
+  // CAS and returns the count); the request's next step claims afresh, so a
+  // step never depends on the SMs an earlier step happened to hold
+  if (kPart && threadIdx.x == 0 && atomicCAS(&S.owner[S.sm], S.tok, 0u) == S.tok)
+    atomicSub(&d->ctl->sm_count, 1u);
 }
 
 // The original kernel: one CTA per VG, hardware block scheduler (Fig. 1a).

@@ -12,6 +12,7 @@
 #include <cuda_runtime.h>
 
 #include <algorithm>
+#include <cmath>
 #include <atomic>
 #include <chrono>
 #include <cstdio>
@@ -35,6 +36,13 @@ using accel::kDescBytes;
 
 constexpr uint32_t kPoolSlots = 16384;      // 4 MiB of descriptors
 constexpr uint32_t kFlagStamps = 1u, kFlagAlive = 2u;  // dispatch.cuh
+constexpr uint32_t kOwnerWords = 1024;     // %smid < 1024 (ids need not be contiguous)
+constexpr uint32_t kFlagProgress = 4u;     // dispatch.cuh: count completed VGs in Ctl::done_vgs
+constexpr int kFairPeriodUs = 150;         // FAIR: feedback period of the monitor
+constexpr double kFairW0 = 16.0;           // FAIR: neutral weight
+constexpr double kFairBeta = 2.0;          // FAIR: weight ~ (slowdown / geometric mean)^beta
+
+bool is_resolve(int policy) { return policy == ACCEL_POLICY_RESOLVE || policy == ACCEL_POLICY_FAIR; }
 
 struct Kernel {
   std::string name;
@@ -42,6 +50,9 @@ struct Kernel {
   const void* prfn;  // accel_persistent<T, RESOLVE>
   const void* nfn;
   const void* tfn;
+  const void* partfn;   // accel_topup<T, PARTITION> (nullptr: not partitionable)
+  int occ_part = 0;     // PARTITION: CTAs per SM (c_i) of partfn
+  uint32_t part_smem = 0;  // PARTITION: dynamic smem padded so c_i CTAs fill the SM
   dim3 block;
   uint32_t dyn_smem;
   uint32_t chunk;
@@ -61,6 +72,7 @@ struct Step {
   uint32_t quota;
   uint32_t first;       // first descriptor (relative to the request's slot)
   uint64_t cov_offset;  // coverage offset of the first launch
+  const uint32_t* order = nullptr;  // dequeue order (device), nullptr = linear
 };
 
 struct Request {
@@ -86,6 +98,13 @@ struct Request {
   uint32_t quota_initial = 0, quota_min = 0, quota_max = 0, resolves = 0;
   uint32_t live = 0;         // RESOLVE: current live quota of the main step
   uint32_t provisioned = 0;  // RESOLVE: main-grid CTAs + sticky top-up CTAs
+  bool part = false;         // PARTITION request
+  uint64_t iso_ns = 0;       // FAIR: isolated-time hint (0: none)
+  uint64_t vgs_hint = 0;     // FAIR: VGs the request runs
+  std::chrono::steady_clock::time_point t_submit;
+  uint32_t done_vgs = 0;     // FAIR: last progress read
+  uint32_t sms = 0;          // PARTITION: current SM quota
+  uint32_t sms_provisioned = 0;  // PARTITION: SMs' worth of CTAs launched for the main step
   bool done = false;
   bool departed_seen = false;  // monitor already re-solved for this departure
   bool fetched = false;
@@ -120,8 +139,11 @@ struct DescHost {
   uint64_t ctl, coverage;
   uint32_t has_prev, pad_a;
   uint64_t trace;
-  uint32_t governed;
-  uint32_t pad0[15];
+  uint32_t governed, tok;
+  uint64_t owner;
+  uint32_t last_step, ctas_per_sm;
+  uint64_t order;
+  uint32_t pad0[8];
   // line 1
   unsigned long long qa;  // alive << 32 | next
   uint32_t pad1[30];
@@ -152,11 +174,13 @@ struct accel_ctx {
   bool epoch_set = false;
   unsigned char* pool = nullptr;
   unsigned char* ctl_pool = nullptr;      // accel::Ctl per descriptor slot
+  uint32_t* owner = nullptr;              // PARTITION: per-SM owner words (kOwnerWords)
   uint32_t* pinned_ring = nullptr;        // staging for live-quota writes
   uint32_t ring_pos = 0;
   std::thread monitor;
   std::atomic<bool> stop{false};
   uint64_t monitor_solves = 0;
+  std::chrono::steady_clock::time_point last_fair{};
   // dispatch variant (env ACCEL_DISPATCH): "" / "dyn" = one dequeue in flight,
   // "dyn2" = two in flight (kCfgDepth2), "stride" = static round robin (ablation)
   uint32_t dispatch_bits = 0;
@@ -283,19 +307,25 @@ int enqueue(accel_ctx* ctx, Request* r) {
   if (r->trace) CK(ctx, cudaMemsetAsync(r->trace, 0, r->trace_elems * sizeof(accel_vg_record), s));
   InitParams p{};
   p.d = ctx->desc_ptr(r->slot);
-  const bool resolve = shared && ctx->cfg.policy == ACCEL_POLICY_RESOLVE;
+  const bool part = shared && r->part;
+  const bool resolve = shared && (is_resolve(ctx->cfg.policy) || part);
   p.ctl = resolve ? ctx->ctl_ptr(r->slot) : nullptr;
-  p.live_init = r->steps[r->main_step].quota;
+  p.live_init = part ? 0xffffffffu : r->steps[r->main_step].quota;
+  p.owner = part ? ctx->owner : nullptr;
+  p.tok = r->slot + 1;
+  p.sm_quota_init = r->sms;
   p.main_step = (uint32_t)r->main_step;
   p.coverage = r->cov;
   p.trace = r->trace;
-  p.flags = kFlagStamps | (shared ? kFlagAlive : 0u);
+  p.flags = kFlagStamps | (shared ? kFlagAlive : 0u) |
+            (shared && ctx->cfg.policy == ACCEL_POLICY_FAIR && r->iso_ns ? kFlagProgress : 0u);
   p.n_steps = (uint32_t)r->steps.size();
   for (size_t j = 0; j < r->steps.size(); ++j) {
     const Step& st = r->steps[j];
     const Kernel& k = ctx->kernels[st.kid];
     p.steps[j] = accel::InitStep{st.first, st.repeat, st.total, st.grid.x, st.grid.y, st.grid.z,
-                                 k.chunk, (uint32_t)st.cov_offset};
+                                 k.chunk, (uint32_t)st.cov_offset, part ? (uint32_t)k.occ_part : 0u,
+                                 shared ? st.order : nullptr};
   }
   CK(ctx, accel::launch_desc_init(p, r->n_desc, s));
   const bool lev = (r->flags & ACCEL_REQ_LAUNCH_EVENTS) != 0;
@@ -306,6 +336,19 @@ int enqueue(accel_ctx* ctx, Request* r) {
   uint32_t li = 0;
   for (const Step& st : r->steps) {
     const Kernel& k = ctx->kernels[st.kid];
+    if (part) {
+      // PARTITION: one sticky grid per step serves all its launches; c_i CTAs
+      // for every SM of the device, so whichever SMs the request gets are
+      // filled (the CTAs on SMs it does not get leave at once)
+      if (lev) CK(ctx, cudaEventRecord(r->ev_launch[li], s));
+      accel::Desc* d = ctx->desc_ptr(r->slot + st.first);
+      uint32_t sticky = st.repeat;
+      void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &sticky};
+      CK(ctx, cudaLaunchKernel(k.partfn, dim3((uint32_t)k.occ_part * (uint32_t)ctx->caps.sms, 1, 1), k.block,
+                               params, k.part_smem, s));
+      li += st.repeat;
+      continue;
+    }
     for (uint32_t l = 0; l < st.repeat; ++l, ++li) {
       if (lev) CK(ctx, cudaEventRecord(r->ev_launch[li], s));
       accel::Desc* d = ctx->desc_ptr(r->slot + st.first + l);
@@ -317,7 +360,7 @@ int enqueue(accel_ctx* ctx, Request* r) {
     }
   }
   if (lev) CK(ctx, cudaEventRecord(r->ev_launch[li], s));
-  if (resolve) CK(ctx, accel::launch_join(ctx->desc_ptr(r->slot + r->n_desc - 1), s));
+  if (resolve) CK(ctx, accel::launch_join(ctx->desc_ptr(r->slot + r->n_desc - 1), part ? kOwnerWords : 0u, s));
   for (const accel_copy& c : r->d2h) CK(ctx, cudaMemcpyAsync(c.dst, c.src, c.bytes, cudaMemcpyDeviceToHost, s));
   CK(ctx, cudaEventRecord(r->ev_done, s));
   return ACCEL_OK;
@@ -333,6 +376,10 @@ int build_request(accel_ctx* ctx, const accel_request& in, std::unique_ptr<Reque
   r->flags = in.flags;
   r->weight = in.weight ? in.weight : 1;
   r->mode = ctx->cfg.mode;
+  r->part = ctx->cfg.mode == ACCEL_MODE_SHARED && ctx->cfg.policy == ACCEL_POLICY_PARTITION;
+  r->iso_ns = in.isolated_ns;
+  r->t_submit = std::chrono::steady_clock::now();
+  if (ctx->cfg.policy == ACCEL_POLICY_FAIR) r->weight = (uint32_t)kFairW0 * r->weight;  // neutral = W0
   uint32_t n_desc = 0;
   uint64_t cov = 0;
   if (in.main_step >= (int32_t)in.n_steps) return ctx->fail(ACCEL_EINVAL, "main_step out of range");
@@ -343,6 +390,8 @@ int build_request(accel_ctx* ctx, const accel_request& in, std::unique_ptr<Reque
     const Kernel& k = ctx->kernels[L.kernel_id];
     if (L.args_size != k.args_size || !L.args) return ctx->fail(ACCEL_EINVAL, "args_size mismatch for " + k.name);
     if (L.repeat < 1) return ctx->fail(ACCEL_EINVAL, "repeat < 1");
+    if (r->part && (!k.partfn || k.occ_part < 1))
+      return ctx->fail(ACCEL_EINVAL, k.name + " has no PARTITION instantiation");
     const uint64_t total = (uint64_t)L.grid.x * L.grid.y * L.grid.z;
     if (total == 0 || total >= 0x7fffffffull || L.grid.y > 65535 || L.grid.z > 65535)
       return ctx->fail(ACCEL_EINVAL, "bad grid");
@@ -352,6 +401,7 @@ int build_request(accel_ctx* ctx, const accel_request& in, std::unique_ptr<Reque
     s.total = (uint32_t)total;
     s.args.assign((const unsigned char*)L.args, (const unsigned char*)L.args + L.args_size);
     s.repeat = L.repeat;
+    s.order = L.order_device;
     s.quota = s.total;
     s.first = n_desc;
     s.cov_offset = cov;
@@ -361,6 +411,11 @@ int build_request(accel_ctx* ctx, const accel_request& in, std::unique_ptr<Reque
     if (in.main_step < 0 && r->steps.back().total > r->steps[r->main_step].total) r->main_step = (int)j;
   }
   r->n_desc = n_desc;
+  {
+    uint64_t vgs = 0;
+    for (const Step& s : r->steps) vgs += (uint64_t)s.total * s.repeat;
+    r->vgs_hint = in.vgs_hint ? in.vgs_hint : vgs;
+  }
   r->cov_elems = ctx->cfg.verify ? cov : 0;
   r->trace_elems = (in.flags & ACCEL_REQ_TRACE) ? cov : 0;
   r->clears.assign(in.clear, in.clear + in.n_clear);
@@ -402,10 +457,76 @@ int apply_quota(accel_ctx* ctx, Request* r, uint32_t q) {
     CK(ctx, cudaEventRecord(ev, ts));
     r->provisioned = q;
   }
+  // the CTAs a shrink evicts leave the running launch: a later growth must top up again
+  if (q < r->live) r->provisioned = std::min(r->provisioned, q);
   r->live = q;
   r->resolves += 1;
   r->quota_min = std::min(r->quota_min, q);
   r->quota_max = std::max(r->quota_max, q);
+  return ACCEL_OK;
+}
+
+// PARTITION: set a running request's SM quota (copy engine).  Shrinking takes
+// effect at its CTAs' next dequeues (part_leave); growing relies on the main
+// grid's CTAs still waiting for an SM and, as insurance, adds a growth grid of
+// c_i CTAs per extra SM (its CTAs that find no SM to claim leave at once).
+int apply_sms(accel_ctx* ctx, Request* r, uint32_t sms) {
+  if (debug_on())
+    std::fprintf(stderr, "[accel] partition req %llu tenant %d sms %u -> %u\n", (unsigned long long)r->id,
+                 r->tenant, r->sms, sms);
+  if (sms == r->sms) return ACCEL_OK;
+  if (cudaEventQuery(r->ev_done) == cudaSuccess) return ACCEL_OK;
+  uint32_t* h = ctx->pinned_ring + (ctx->ring_pos++ % kRing);
+  *h = sms;
+  CK(ctx, cudaMemcpyAsync(ctx->ctl_pool + (size_t)r->slot * kCtlBytes + 8 /* Ctl::sm_quota */, h,
+                          sizeof(uint32_t), cudaMemcpyHostToDevice, ctx->ctl));
+  if (sms > r->sms_provisioned) {
+    const Step& st = r->steps[r->main_step];
+    const Kernel& k = ctx->kernels[st.kid];
+    accel::Desc* d = ctx->desc_ptr(r->slot + st.first);
+    uint32_t sticky = st.repeat;
+    void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &sticky};
+    cudaStream_t ts = ctx->topup[ctx->topup_rr++ % accel_ctx::kTopupStreams];
+    CK(ctx, cudaLaunchKernel(k.partfn, dim3((sms - r->sms_provisioned) * (uint32_t)k.occ_part, 1, 1), k.block,
+                             params, k.part_smem, ts));
+    cudaEvent_t ev;
+    CK(ctx, ctx->get_event(&ev));
+    r->ev_topups.push_back(ev);
+    CK(ctx, cudaEventRecord(ev, ts));
+    r->sms_provisioned = sms;
+  }
+  const uint32_t c = (uint32_t)ctx->kernels[r->steps[r->main_step].kid].occ_part;
+  r->sms = sms;
+  r->live = sms * c;
+  r->resolves += 1;
+  r->quota_min = std::min(r->quota_min, sms * c);
+  r->quota_max = std::max(r->quota_max, sms * c);
+  return ACCEL_OK;
+}
+
+int assign_sms(accel_ctx* ctx, const std::vector<Request*>& order, size_t first_new) {
+  std::vector<accel_demand> ds(order.size());
+  for (size_t i = 0; i < order.size(); ++i) {
+    Request* r = order[i];
+    int rc = demand_for(ctx, r->steps[r->main_step], r->weight, &ds[i]);
+    if (rc) return ctx->fail(rc, "kernel does not fit on an SM");
+  }
+  std::vector<uint32_t> sms(order.size()), per(order.size());
+  int rc = accel_solve_sms(&ctx->caps, ds.data(), (int32_t)ds.size(), sms.data(), per.data());
+  if (rc) return ctx->fail(rc, "accel_solve_sms failed");
+  ctx->monitor_solves += 1;
+  for (size_t i = 0; i < first_new; ++i) {
+    rc = apply_sms(ctx, order[i], sms[i]);
+    if (rc) return rc;
+  }
+  for (size_t i = first_new; i < order.size(); ++i) {
+    Request* r = order[i];
+    const uint32_t c = (uint32_t)ctx->kernels[r->steps[r->main_step].kid].occ_part;
+    for (Step& st : r->steps) st.quota = sms[i] * (uint32_t)ctx->kernels[st.kid].occ_part;
+    r->sms = r->sms_provisioned = sms[i];
+    r->quota_initial = r->quota_min = r->quota_max = sms[i] * c;
+    r->live = r->provisioned = sms[i] * c;
+  }
   return ACCEL_OK;
 }
 
@@ -422,6 +543,7 @@ int assign_quotas(accel_ctx* ctx, std::vector<std::unique_ptr<Request>>& fresh) 
   }
   for (auto& r : fresh) order.push_back(r.get());
   if (order.empty()) return ACCEL_OK;
+  if (ctx->cfg.policy == ACCEL_POLICY_PARTITION) return assign_sms(ctx, order, order.size() - fresh.size());
   std::vector<accel_demand> ds(order.size());
   for (size_t i = 0; i < order.size(); ++i) {
     Request* r = order[i];
@@ -433,7 +555,7 @@ int assign_quotas(accel_ctx* ctx, std::vector<std::unique_ptr<Request>>& fresh) 
   if (rc) return ctx->fail(rc, "accel_solve failed");
   ctx->monitor_solves += 1;
   const size_t first_new = order.size() - fresh.size();
-  if (ctx->cfg.policy == ACCEL_POLICY_RESOLVE)
+  if (is_resolve(ctx->cfg.policy))
     for (size_t i = 0; i < first_new; ++i) {
       rc = apply_quota(ctx, order[i], q[i]);
       if (rc) return rc;
@@ -469,6 +591,56 @@ int assign_quotas(accel_ctx* ctx, std::vector<std::unique_ptr<Request>>& fresh) 
   return ACCEL_OK;
 }
 
+// FAIR (DESIGN.md R-fair-1..3): read every running request's completed VGs,
+// estimate its slowdown so far, sigma_i = elapsed_i / (progress_i * T_iso_i),
+// and set weight_i = W0 * (sigma_i / geomean sigma)^beta, clamped.  Returns
+// true when a weight moved by more than 25 % (then the caller re-solves).
+bool fair_weights(accel_ctx* ctx) {
+  std::vector<Request*> rs;
+  for (auto& kv : ctx->reqs) {
+    Request* r = kv.second.get();
+    if (r->mode == ACCEL_MODE_SHARED && !r->done && r->iso_ns && r->vgs_hint) rs.push_back(r);
+  }
+  if (rs.size() < 2) return false;
+  uint32_t* h = ctx->pinned_ring + (ctx->ring_pos % kRing);
+  ctx->ring_pos += (uint32_t)rs.size();
+  if (ctx->ring_pos % kRing < rs.size()) return false;  // wrap: skip this round
+  for (size_t i = 0; i < rs.size(); ++i)
+    if (ctx->cuda(cudaMemcpyAsync(h + i, ctx->ctl_pool + (size_t)rs[i]->slot * kCtlBytes + 16 /* done_vgs */,
+                                  sizeof(uint32_t), cudaMemcpyDeviceToHost, ctx->ctl),
+                  "cudaMemcpyAsync(progress)"))
+      return false;
+  if (ctx->cuda(cudaStreamSynchronize(ctx->ctl), "cudaStreamSynchronize(ctl)")) return false;
+  const auto now = std::chrono::steady_clock::now();
+  std::vector<double> sig(rs.size(), 0.0);
+  int n = 0;
+  for (size_t i = 0; i < rs.size(); ++i) {
+    Request* r = rs[i];
+    r->done_vgs = h[i];
+    const double el = (double)std::chrono::duration_cast<std::chrono::nanoseconds>(now - r->t_submit).count();
+    const double p = std::min(1.0, (double)r->done_vgs / (double)r->vgs_hint);
+    if (p < 0.01 || el < 0.05 * (double)r->iso_ns) continue;  // too early to tell
+    sig[i] = el / (p * (double)r->iso_ns);
+    ++n;
+  }
+  if (n < 2) return false;
+  std::vector<uint32_t> w(rs.size());
+  accel_fair_weights(sig.data(), (int32_t)rs.size(), w.data());
+  bool moved = false;
+  for (size_t i = 0; i < rs.size(); ++i) {
+    if (sig[i] <= 0.0) continue;
+    const uint32_t wi = w[i];
+    if (wi * 4 > rs[i]->weight * 5 || wi * 5 < rs[i]->weight * 4) moved = true;
+    rs[i]->weight = wi;
+  }
+  if (moved && debug_on()) {
+    std::fprintf(stderr, "[accel] fair:");
+    for (size_t i = 0; i < rs.size(); ++i) std::fprintf(stderr, " t%d s=%.2f w=%u", rs[i]->tenant, sig[i], rs[i]->weight);
+    std::fprintf(stderr, "\n");
+  }
+  return moved;
+}
+
 // Host monitor (RESOLVE): detects departures without host synchronisation by
 // polling the requests' completion events, and re-solves the survivors.
 void monitor_loop(accel_ctx* ctx) {
@@ -478,7 +650,7 @@ void monitor_loop(accel_ctx* ctx) {
     std::this_thread::sleep_for(std::chrono::microseconds(busy ? 20 : 500));
     std::unique_lock<std::mutex> g(ctx->mu);
     busy = false;
-    if (ctx->poisoned || ctx->cfg.mode != ACCEL_MODE_SHARED || ctx->cfg.policy != ACCEL_POLICY_RESOLVE)
+    if (ctx->poisoned || ctx->cfg.mode != ACCEL_MODE_SHARED || ctx->cfg.policy == ACCEL_POLICY_STATIC)
       continue;
     bool departed = false, running = false;
     for (auto& kv : ctx->reqs) {
@@ -494,7 +666,15 @@ void monitor_loop(accel_ctx* ctx) {
     }
     busy = running;
     if (departed && debug_on()) std::fprintf(stderr, "[accel] monitor: departure (running=%d)\n", (int)running);
-    if (departed && running) {
+    bool resolve_now = departed && running;
+    if (running && ctx->cfg.policy == ACCEL_POLICY_FAIR) {
+      const auto now = std::chrono::steady_clock::now();
+      if (now - ctx->last_fair >= std::chrono::microseconds(kFairPeriodUs)) {
+        ctx->last_fair = now;
+        if (fair_weights(ctx)) resolve_now = true;
+      }
+    }
+    if (resolve_now) {
       std::vector<std::unique_ptr<Request>> none;
       assign_quotas(ctx, none);
     }
@@ -552,6 +732,23 @@ void release_request(accel_ctx* ctx, Request* r) {
 
 extern "C" {
 
+int accel_fair_weights(const double* slowdown, int32_t k, uint32_t* weight_out) {
+  if (k < 0 || (k > 0 && (!slowdown || !weight_out))) return ACCEL_EINVAL;
+  double lsum = 0.0;
+  int n = 0;
+  for (int i = 0; i < k; ++i)
+    if (slowdown[i] > 0.0) {
+      lsum += std::log(slowdown[i]);
+      ++n;
+    }
+  const double gm = n ? std::exp(lsum / n) : 1.0;
+  for (int i = 0; i < k; ++i) {
+    const double w = slowdown[i] > 0.0 ? kFairW0 * std::pow(slowdown[i] / gm, kFairBeta) : kFairW0;
+    weight_out[i] = (uint32_t)std::lround(std::min(1024.0, std::max(1.0, w)));
+  }
+  return ACCEL_OK;
+}
+
 const char* accel_last_error(const accel_ctx* ctx) {
   return ctx ? ctx->err.c_str() : g_init_error.c_str();
 }
@@ -559,7 +756,9 @@ const char* accel_last_error(const accel_ctx* ctx) {
 int accel_init(const accel_config* cfg, accel_ctx** out) {
   if (!cfg || !out) return ACCEL_EINVAL;
   if (cfg->mode != ACCEL_MODE_NATIVE && cfg->mode != ACCEL_MODE_SHARED) return ACCEL_EINVAL;
-  if (cfg->policy != ACCEL_POLICY_STATIC && cfg->policy != ACCEL_POLICY_RESOLVE) return ACCEL_EINVAL;
+  if (cfg->policy != ACCEL_POLICY_STATIC && cfg->policy != ACCEL_POLICY_RESOLVE &&
+      cfg->policy != ACCEL_POLICY_PARTITION && cfg->policy != ACCEL_POLICY_FAIR)
+    return ACCEL_EINVAL;
   auto ctx = std::make_unique<accel_ctx>();
   ctx->cfg = *cfg;
   auto init_fail = [&](cudaError_t e, const char* what) {
@@ -586,6 +785,10 @@ int accel_init(const accel_config* cfg, accel_ctx** out) {
     return init_fail(e, "cudaMalloc(pool)");
   if ((e = cudaMalloc(&ctx->ctl_pool, (size_t)kPoolSlots * kCtlBytes)) != cudaSuccess)
     return init_fail(e, "cudaMalloc(ctl)");
+  if ((e = cudaMalloc(&ctx->owner, kOwnerWords * sizeof(uint32_t))) != cudaSuccess)
+    return init_fail(e, "cudaMalloc(owner)");
+  if ((e = cudaMemset(ctx->owner, 0, kOwnerWords * sizeof(uint32_t))) != cudaSuccess)
+    return init_fail(e, "cudaMemset(owner)");
   if ((e = cudaHostAlloc(reinterpret_cast<void**>(&ctx->pinned_ring), kRing * sizeof(uint32_t),
                          cudaHostAllocDefault)) != cudaSuccess)
     return init_fail(e, "cudaHostAlloc(ring)");
@@ -620,6 +823,7 @@ int accel_finalize(accel_ctx* ctx) {
   if (ctx->epoch) cudaEventDestroy(ctx->epoch);
   if (ctx->pool) cudaFree(ctx->pool);
   if (ctx->ctl_pool) cudaFree(ctx->ctl_pool);
+  if (ctx->owner) cudaFree(ctx->owner);
   if (ctx->pinned_ring) cudaFreeHost(ctx->pinned_ring);
   delete ctx;
   return ACCEL_OK;
@@ -630,7 +834,9 @@ int accel_set_mode(accel_ctx* ctx, int32_t mode, int32_t policy) {
   std::lock_guard<std::mutex> g(ctx->mu);
   if (ctx->poisoned) return ACCEL_ESTATE;
   if (mode != ACCEL_MODE_NATIVE && mode != ACCEL_MODE_SHARED) return ctx->fail(ACCEL_EINVAL, "bad mode");
-  if (policy != ACCEL_POLICY_STATIC && policy != ACCEL_POLICY_RESOLVE) return ctx->fail(ACCEL_EINVAL, "bad policy");
+  if (policy != ACCEL_POLICY_STATIC && policy != ACCEL_POLICY_RESOLVE && policy != ACCEL_POLICY_PARTITION &&
+      policy != ACCEL_POLICY_FAIR)
+    return ctx->fail(ACCEL_EINVAL, "bad policy");
   for (auto& kv : ctx->reqs) {
     int rc = refresh_done(ctx, kv.second.get());
     if (rc) return rc;
@@ -652,6 +858,7 @@ int accel_kernel_register(accel_ctx* ctx, const accel_kernel_desc* d, int32_t* k
   k.prfn = d->persistent_resolve_fn ? d->persistent_resolve_fn : d->persistent_fn;
   k.nfn = d->native_fn;
   k.tfn = d->topup_fn ? d->topup_fn : d->persistent_fn;
+  k.partfn = d->partition_fn;
   k.block = dim3(d->block.x, d->block.y ? d->block.y : 1, d->block.z ? d->block.z : 1);
   k.dyn_smem = d->dyn_smem;
   k.chunk = d->chunk ? d->chunk : 1;
@@ -673,6 +880,39 @@ int accel_kernel_register(accel_ctx* ctx, const accel_kernel_desc* d, int32_t* k
   }
   CK(ctx, cudaOccupancyMaxActiveBlocksPerMultiprocessor(&k.occ_p, k.pfn, (int)k.threads(), k.dyn_smem));
   CK(ctx, cudaOccupancyMaxActiveBlocksPerMultiprocessor(&k.occ_n, k.nfn, (int)k.threads(), k.dyn_smem));
+  if (k.partfn) {
+    // PARTITION: c_i CTAs alone on an SM, then pad the dynamic shared memory so
+    // that exactly c_i of them take all of it (1 KiB reserved per CTA, 128-B
+    // granules): no CTA of another kernel fits on an SM the request holds
+    CK(ctx, cudaFuncSetAttribute(k.partfn, cudaFuncAttributePreferredSharedMemoryCarveout, 100));
+    if (k.dyn_smem > 48 * 1024)
+      CK(ctx, cudaFuncSetAttribute(k.partfn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)k.dyn_smem));
+    cudaFuncAttributes pa;
+    CK(ctx, cudaFuncGetAttributes(&pa, k.partfn));
+    CK(ctx, cudaOccupancyMaxActiveBlocksPerMultiprocessor(&k.occ_part, k.partfn, (int)k.threads(), k.dyn_smem));
+    int sm_smem = 0, max_optin = 0;
+    CK(ctx, cudaDeviceGetAttribute(&sm_smem, cudaDevAttrMaxSharedMemoryPerMultiprocessor, ctx->cfg.device));
+    CK(ctx, cudaDeviceGetAttribute(&max_optin, cudaDevAttrMaxSharedMemoryPerBlockOptin, ctx->cfg.device));
+    k.part_smem = k.dyn_smem;
+    if (k.occ_part >= 1) {
+      int64_t per = (int64_t)(sm_smem / k.occ_part) / 128 * 128;  // footprint per CTA
+      for (; per >= 128; per -= 128) {
+        const int64_t dyn = per - 1024 - (int64_t)pa.sharedSizeBytes;
+        if (dyn < (int64_t)k.dyn_smem) break;
+        if (dyn + (int64_t)pa.sharedSizeBytes > max_optin) continue;
+        CK(ctx, cudaFuncSetAttribute(k.partfn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)dyn));
+        int occ = 0;
+        CK(ctx, cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k.partfn, (int)k.threads(), (size_t)dyn));
+        if (occ == k.occ_part) {
+          k.part_smem = (uint32_t)dyn;
+          break;
+        }
+      }
+      if (k.part_smem > 48 * 1024 || k.dyn_smem > 48 * 1024)
+        CK(ctx, cudaFuncSetAttribute(k.partfn, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                     (int)std::max(k.part_smem, k.dyn_smem)));
+    }
+  }
   accel_demand dem;
   int rc = accel_demand_of(&ctx->caps, k.threads(), (uint32_t)k.num_regs,
                            (uint32_t)(k.static_smem + k.dyn_smem), 1, 1, &dem);
@@ -699,6 +939,8 @@ int accel_kernel_info_get(accel_ctx* ctx, int32_t kernel_id, accel_kernel_info* 
   out->static_smem = k.static_smem;
   out->occ_persistent = k.occ_p;
   out->occ_native = k.occ_n;
+  out->occ_partition = k.occ_part;
+  out->partition_smem = k.part_smem;
   return ACCEL_OK;
 }
 
@@ -830,6 +1072,18 @@ int accel_launch_times(accel_ctx* ctx, uint64_t request_id, float* ms_out, uint3
   if (!r->done) return ACCEL_ENOTREADY;
   if (r->ev_launch.empty()) return ctx->fail(ACCEL_EINVAL, "request had no ACCEL_REQ_LAUNCH_EVENTS");
   const uint32_t m = std::min<uint32_t>(n, r->n_desc);
+  if (r->part) {
+    // PARTITION: one grid per step, events around it; a launch gets the
+    // step's time divided by its launches
+    for (const Step& st : r->steps) {
+      const uint32_t end = st.first + st.repeat;
+      float ms = 0.f;
+      CK(ctx, cudaEventElapsedTime(&ms, r->ev_launch[st.first], r->ev_launch[end]));
+      for (uint32_t i = st.first; i < end && i < m; ++i) ms_out[i] = ms / (float)st.repeat;
+    }
+    *n_out = m;
+    return ACCEL_OK;
+  }
   for (uint32_t i = 0; i < m; ++i)
     CK(ctx, cudaEventElapsedTime(&ms_out[i], r->ev_launch[i], r->ev_launch[i + 1]));
   *n_out = m;

@@ -28,6 +28,9 @@ __global__ void desc_init_kernel(const InitParams p, uint32_t n_desc) {
   if (i == 0 && p.ctl != nullptr) {
     p.ctl->live = p.live_init;
     p.ctl->cur = 0;
+    p.ctl->sm_quota = p.sm_quota_init;
+    p.ctl->sm_count = 0;
+    p.ctl->done_vgs = 0;
   }
   if (i >= n_desc) return;
   uint32_t s = 0;
@@ -46,7 +49,12 @@ __global__ void desc_init_kernel(const InitParams p, uint32_t n_desc) {
   d->ctl = p.ctl;
   d->coverage = p.coverage ? p.coverage + st.cov_offset + (size_t)r * st.total : nullptr;
   d->trace = p.trace ? p.trace + st.cov_offset + (size_t)r * st.total : nullptr;
-  d->governed = s == p.main_step ? 1u : 0u;
+  d->governed = (s == p.main_step && p.owner == nullptr) ? 1u : 0u;
+  d->tok = p.tok;
+  d->owner = p.owner;
+  d->last_step = s + 1 == p.n_steps ? 1u : 0u;
+  d->ctas_per_sm = st.ctas_per_sm;
+  d->order = st.order;
   d->t_first = ULLONG_MAX;
   d->t_last = 0;
   d->ctas_started = 0;
@@ -55,18 +63,27 @@ __global__ void desc_init_kernel(const InitParams p, uint32_t n_desc) {
   d->evicted = 0;
   d->draining = 0;
   d->last_live = 0;
-  d->topped = 0;
+  d->topped = p.owner != nullptr ? 1u : 0u;   // PARTITION: any grid may serve any launch
   d->req_idx = i;
   d->has_prev = i > 0 ? 1u : 0u;
   d->qa = 0;
 }
 
-__global__ void join_kernel(const Desc* last) {
+// Request completion: wait until the last launch completed if another grid
+// may still be serving it.  PARTITION: then hand back every SM the request
+// still owns (a safety net: its CTAs free their SMs when they finish).
+__global__ void join_kernel(const Desc* last, uint32_t nsm) {
   if (threadIdx.x == 0 && ld_volatile(&last->topped)) wait_complete(last);
+  __syncwarp();
+  if (last->owner != nullptr)
+    for (uint32_t sm = threadIdx.x; sm < nsm; sm += 32) {
+      const uint32_t o = ld_volatile(&last->owner[sm]);
+      if ((o & ~(kOwnRel | kOwnClaim)) == last->tok) atomicCAS(&last->owner[sm], o, 0u);
+    }
 }
 
-cudaError_t launch_join(const Desc* last, cudaStream_t s) {
-  join_kernel<<<1, 32, 0, s>>>(last);
+cudaError_t launch_join(const Desc* last, uint32_t nsm, cudaStream_t s) {
+  join_kernel<<<1, 32, 0, s>>>(last, nsm);
   return cudaGetLastError();
 }
 
@@ -84,7 +101,8 @@ accel_kernel_desc make_desc(const char* name) {
   d.persistent_fn = reinterpret_cast<const void*>(&accel_persistent<T, false>);
   d.persistent_resolve_fn = reinterpret_cast<const void*>(&accel_persistent<T, true>);
   d.native_fn = reinterpret_cast<const void*>(&accel_native<T>);
-  d.topup_fn = reinterpret_cast<const void*>(&accel_topup<T>);
+  d.topup_fn = reinterpret_cast<const void*>(&accel_topup<T, false>);
+  d.partition_fn = reinterpret_cast<const void*>(&accel_topup<T, true>);
   d.block = accel_dim3{(uint32_t)T::kThreads, 1u, 1u};
   d.dyn_smem = T::kDynSmem;
   d.regs = 0;

@@ -51,6 +51,7 @@ class Step:
     grid: tuple[int, int, int]
     args: C.Structure
     repeat: int = 1
+    order: torch.Tensor | None = None   # dequeue order (device uint32 permutation), None = linear
 
 
 @dataclass
@@ -68,6 +69,9 @@ class Job:
         self._pinned_in: dict[str, torch.Tensor] = {}
         self._pinned_out: dict[str, torch.Tensor] = {}
         self.main_step = -1  # -1: the library picks the step with the most VGs
+        # FAIR policy: completed VGs / static VGs tracks progress (False for
+        # dynamic-total kernels, bfs: they run fewer VGs than their grids)
+        self.progress_hint = True
 
     # ---- e2e: host buffers ----------------------------------------------
     def pin_host(self) -> None:
@@ -96,7 +100,8 @@ class Job:
         keep = []
         for i, s in enumerate(self.steps):
             steps[i] = abi.accel_launch(kernel_ids[s.kernel], abi.accel_dim3(*s.grid),
-                                        C.cast(C.pointer(s.args), C.c_void_p), C.sizeof(s.args), s.repeat)
+                                        C.cast(C.pointer(s.args), C.c_void_p), C.sizeof(s.args), s.repeat,
+                                        s.order.data_ptr() if s.order is not None else None)
             keep.append(s.args)
         clears = (abi.accel_clear * max(1, len(self.clears)))()
         for i, (t, v) in enumerate(self.clears):
@@ -215,6 +220,7 @@ class BfsJob(Job):
 
     def __init__(self, d: dict, device="cuda", levels: int | None = None):
         super().__init__(name="bfs", device=torch.device(device))
+        self.progress_hint = False
         self.nv, self.ne, self.src = d["nv"], d["ne"], d["src"]
         self.levels = levels or d.get("levels", 24)
         self.inputs = {"row_ptr": _dev(d["row_ptr"], self.device), "col": _dev(d["col"], self.device)}
@@ -239,6 +245,60 @@ class BfsJob(Job):
         return {"bytes": b, "bytes_per_launch": b / self.levels, "bound": "hbm", "launches": self.levels}
 
 
+# ---- dequeue order (accel_launch.order_device): most expensive VGs first ----
+# The software queue hands out VGs in any order (DESIGN.md R-disp-7); ordering
+# them by decreasing estimated cost is longest-processing-time-first list
+# scheduling over the persistent CTAs: the last VGs dealt are the cheapest, so
+# the tail after the queue runs dry is short.  These are scheduling hints
+# computed from the inputs' shape, not results; NATIVE mode ignores them.
+def _lpt_order(cost: np.ndarray, device) -> torch.Tensor:
+    order = np.argsort(-np.asarray(cost, dtype=np.float64), kind="stable").astype(np.int32)
+    return torch.from_numpy(order).to(device)
+
+
+def _cutcp_vg_cost(d: dict, grid) -> np.ndarray:
+    """Atoms a cutcp VG streams: the cell rows and trimmed x-ranges its body
+    walks (tenants/cutcp.cuh), counted from the cell index."""
+    gx, gy, gz = grid
+    h, cs, nc = float(d["h"]), float(d["cell"]), int(d["ncell_1d"])
+    cm = float(d["cutoff"]) + 0.05
+    cst = np.asarray(d["cell_start"], dtype=np.int64)
+    vx, vy, vz = np.meshgrid(np.arange(gx), np.arange(gy), np.arange(gz), indexing="xy")
+    vx, vy, vz = (a.transpose(2, 0, 1).ravel() for a in (vx, vy, vz))   # x fastest
+    b0 = [h * 8 * v for v in (vx, vy, vz)]
+    b1 = [h * (8 * v + 7) for v in (vx, vy, vz)]
+    cl = lambda v: np.clip(v, 0, nc - 1)  # noqa: E731
+    cy0, cy1 = cl(np.floor((b0[1] - cm) / cs).astype(int)), cl(np.floor((b1[1] + cm) / cs).astype(int))
+    cz0, cz1 = cl(np.floor((b0[2] - cm) / cs).astype(int)), cl(np.floor((b1[2] + cm) / cs).astype(int))
+    cost = np.zeros(vx.size)
+    gap = lambda lo, hi, c: np.maximum(0.0, np.maximum(c * cs - hi, lo - (c + 1) * cs))  # noqa: E731
+    for dz in range(int((cz1 - cz0).max()) + 1):
+        cz = cz0 + dz
+        okz = cz <= cz1
+        gzv = gap(b0[2], b1[2], cz)
+        for dy in range(int((cy1 - cy0).max()) + 1):
+            cy = cy0 + dy
+            ok = okz & (cy <= cy1)
+            gyv = gap(b0[1], b1[1], cy)
+            d2 = gyv * gyv + gzv * gzv
+            ok &= d2 < cm * cm
+            rx = np.sqrt(np.maximum(cm * cm - d2, 0.0))
+            cx0 = cl(np.floor((b0[0] - rx) / cs).astype(int))
+            cx1 = cl(np.floor((b1[0] + rx) / cs).astype(int))
+            row = (np.minimum(cz, nc - 1) * nc + np.minimum(cy, nc - 1)) * nc
+            cost += np.where(ok, cst[row + cx1 + 1] - cst[row + cx0], 0)
+    return cost
+
+
+def _tpacf_vg_cost(n: int, S: int, grid) -> np.ndarray:
+    """Q tiles a tpacf VG (x, y) walks: DD / RR blocks (y <= S) start at their
+    diagonal tile, DR blocks (y > S) walk all of them."""
+    gx, gy, _ = grid
+    x = np.tile(np.arange(gx), gy)
+    y = np.repeat(np.arange(gy), gx)
+    return np.where(y <= S, gx - x - 0.5, gx).astype(np.float64)
+
+
 class CutcpJob(Job):
     def __init__(self, d: dict, device="cuda"):
         super().__init__(name="cutcp", device=torch.device(device))
@@ -251,7 +311,8 @@ class CutcpJob(Job):
         self.args = abi.accel_cutcp_args(self.inputs["atoms"].data_ptr(), self.inputs["cell_start"].data_ptr(),
                                          d["ncell_1d"], d["cell"], self.nx, self.ny, self.nz, d["h"],
                                          d["cutoff"], d["excl"], self.v.data_ptr())
-        self.steps = [Step("cutcp", (_cdiv(self.nx, 8), _cdiv(self.ny, 8), _cdiv(self.nz, 8)), self.args, 1)]
+        grid = (_cdiv(self.nx, 8), _cdiv(self.ny, 8), _cdiv(self.nz, 8))
+        self.steps = [Step("cutcp", grid, self.args, 1, _lpt_order(_cutcp_vg_cost(d, grid), self.device))]
 
     def result(self):
         return {"v": _np(self.v, np.float32).reshape(self.nz, self.ny, self.nx)}
@@ -280,7 +341,8 @@ class TpacfJob(Job):
                                          self.inputs["binb"].data_ptr(), self.n, self.S, self.nedges,
                                          p, p + 8 * nb, p + 16 * nb)
         self.clears = [(self.hists, 0)]
-        self.steps = [Step("tpacf", (_cdiv(self.n, 256), 2 * self.S + 1, 1), self.args, 1)]
+        grid = (_cdiv(self.n, 256), 2 * self.S + 1, 1)
+        self.steps = [Step("tpacf", grid, self.args, 1, _lpt_order(_tpacf_vg_cost(self.n, self.S, grid), self.device))]
 
     def result(self):
         h = _np(self.hists, np.uint64).reshape(3, -1)

@@ -42,7 +42,9 @@ from paper_conf_cgo_margiolaso16_b200.runtime import Accel  # noqa: E402
 
 TENANTS = ["bfs", "cutcp", "stencil", "tpacf", "histo", "spmv", "sgemm", "mriq"]
 MODES = [("native", abi.MODE_NATIVE, abi.POLICY_STATIC), ("resolve", abi.MODE_SHARED, abi.POLICY_RESOLVE),
-         ("static", abi.MODE_SHARED, abi.POLICY_STATIC)]
+         ("static", abi.MODE_SHARED, abi.POLICY_STATIC), ("partition", abi.MODE_SHARED, abi.POLICY_PARTITION),
+         ("fair", abi.MODE_SHARED, abi.POLICY_FAIR)]
+SHARED = ["resolve", "static", "partition", "fair"]
 
 
 def gm(xs):
@@ -58,6 +60,7 @@ class Runner:
         self.jobs = {t: [make_job(t, synth.preset(t, size, seed=11 + i), dev) for i in range(2)]
                      for t in tenants}
         self.flush_buf = torch.empty(256 * 1024 * 1024 // 4, dtype=torch.float32, device=dev)
+        self.ta = {}   # FAIR hints: isolated native times per tenant
 
     def set(self, mode, policy):
         if self.acc.mode != mode or self.acc.policy != policy:
@@ -70,14 +73,15 @@ class Runner:
         torch.cuda.synchronize()
         self.acc.epoch()
         ids = []
+        iso = [self.ta.get(j.name, 0.0) for j in jobs] if policy == abi.POLICY_FAIR else None
         if delays_s is None:
-            ids = self.acc.submit(jobs, tenants=list(range(len(jobs))))
+            ids = self.acc.submit(jobs, tenants=list(range(len(jobs))), isolated_ms=iso)
         else:
             t0 = time.perf_counter()
             for i, (j, dl) in enumerate(zip(jobs, delays_s)):
                 while time.perf_counter() - t0 < dl:
                     pass
-                ids += self.acc.submit([j], tenants=[i])
+                ids += self.acc.submit([j], tenants=[i], isolated_ms=None if iso is None else [iso[i]])
         self.acc.sync()
         st = [self.acc.stats(i) for i in ids]
         self.acc.release()
@@ -99,9 +103,9 @@ def mix_metrics(st, ta_list):
             "WANTT": max(t / a for t, a in zip(ts, ta_list)), "ts_ms": ts}
 
 
-def config3(r: Runner, ta, reps):
+def config3(r: Runner, ta, reps, only=None):
     mixes = []
-    for a, b in itertools.product(TENANTS, TENANTS):
+    for a, b in (only or itertools.product(TENANTS, TENANTS)):
         ja = r.jobs[a][0]
         jb = r.jobs[b][1] if a == b else r.jobs[b][0]
         res = {"mix": [a, b]}
@@ -112,7 +116,7 @@ def config3(r: Runner, ta, reps):
         print(json.dumps({"mix": res["mix"], **{n: {k: round(v, 3) for k, v in res[n].items()} for n, _, _ in MODES}}),
               flush=True)
     out = {}
-    for name in ("resolve", "static"):
+    for name in SHARED:
         fi = [m["native"]["U"] / m[name]["U"] for m in mixes]
         stp = [m[name]["STP"] / m["native"]["STP"] for m in mixes]
         thr = [m["native"]["makespan_ms"] / m[name]["makespan_ms"] for m in mixes]
@@ -141,7 +145,7 @@ def config4(r: Runner, ta, reps):
                                                   for i in range(len(order))]))
         print(name, json.dumps({k: (round(v, 3) if isinstance(v, float) else v) for k, v in out[name].items()}),
               flush=True)
-    for name in ("resolve", "static"):
+    for name in SHARED:
         out[name]["FI"] = out["native"]["U"] / out[name]["U"]
         out[name]["STP_ratio"] = out[name]["STP"] / out["native"]["STP"]
         out[name]["throughput_speedup"] = out["native"]["makespan_ms"] / out[name]["makespan_ms"]
@@ -162,7 +166,7 @@ def sampled(r: Runner, ta, reps, k, n, seed):
             res[name] = {kk: statistics.mean(x[kk] for x in runs) for kk in ("U", "STP", "ANTT", "makespan_ms", "WANTT")}
         mixes.append(res)
     out = {}
-    for name in ("resolve", "static"):
+    for name in SHARED:
         fi = [m["native"]["U"] / m[name]["U"] for m in mixes]
         out[name] = {"U_gmean": gm([m[name]["U"] for m in mixes]), "FI_gmean": gm(fi),
                      "FI_min": min(fi), "FI_max": max(fi),
@@ -185,18 +189,29 @@ def main():
     ap.add_argument("--reps", type=int, default=3)
     ap.add_argument("--size", default="default")
     ap.add_argument("--out", default=None)
+    ap.add_argument("--only", default=None, help="c3: comma-separated a:b pairs, e.g. mriq:mriq,cutcp:sgemm")
+    ap.add_argument("--tenants", default=None, help="restrict the tenants loaded (comma-separated)")
+    ap.add_argument("--modes", default=None, help="restrict the modes (comma-separated; native is always run)")
     a = ap.parse_args()
     dev = torch.device("cuda", 0)
+    if a.tenants:
+        TENANTS[:] = a.tenants.split(",")
+    if a.modes:
+        keep = set(a.modes.split(",")) | {"native"}
+        MODES[:] = [m for m in MODES if m[0] in keep]
+        SHARED[:] = [n for n in SHARED if n in keep]
     r = Runner(TENANTS, a.size, dev)
     # warm every tenant in every mode once (module load, first touch)
     for t, (j, _) in r.jobs.items():
         for _, mode, pol in MODES:
             r.run([j], mode, pol)
     ta = r.isolated(max(3, a.reps))
+    r.ta = dict(ta)
     print("T(a) ms", json.dumps({k: round(v, 3) for k, v in ta.items()}), flush=True)
     res = {"config": a.config, "size": a.size, "reps": a.reps, "T_a_ms": ta}
     if a.config == "c3":
-        mixes, summ = config3(r, ta, a.reps)
+        only = [tuple(p.split(":")) for p in a.only.split(",")] if a.only else None
+        mixes, summ = config3(r, ta, a.reps, only)
         res.update({"mixes": mixes, "summary": summ})
         print("SUMMARY", json.dumps(summ), flush=True)
     elif a.config == "f2":

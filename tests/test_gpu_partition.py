@@ -1,0 +1,157 @@
+"""GPU: the PARTITION policy (whole SMs per request, DESIGN.md R-part-*):
+every tenant stays exact (== the native launch of the same body, == the
+oracle) and covers every VG once, alone, in mixes, with SMs handed over on
+arrival and departure; concurrent requests do not share SMs."""
+import time
+
+import numpy as np
+import pytest
+
+import synth
+from tests.gpu_util import assert_close_fp32
+
+pytestmark = pytest.mark.gpu
+
+TENANTS = ["mop", "stencil", "histo", "bfs", "cutcp", "tpacf", "spmv", "sgemm", "mriq"]
+
+
+def _acc(caps=None):
+    import torch
+    if not torch.cuda.is_available():
+        pytest.skip("no GPU")
+    from paper_conf_cgo_margiolaso16_b200 import abi
+    from paper_conf_cgo_margiolaso16_b200.runtime import Accel
+    return Accel(device=0, mode=abi.MODE_SHARED, policy=abi.POLICY_PARTITION, verify=True,
+                 caps=abi.accel_caps(*caps) if caps else None)
+
+
+@pytest.fixture(scope="module")
+def pacc():
+    a = _acc()
+    yield a
+    a.close()
+
+
+@pytest.fixture(scope="module")
+def pacc_2sm():
+    a = _acc((2, 2048, 65536, 233472, 32))   # the solver sees 2 SMs: many VGs per CTA
+    yield a
+    a.close()
+
+
+def _native_then_partition(acc, make):
+    from paper_conf_cgo_margiolaso16_b200 import abi
+    out = {}
+    for mode in (abi.MODE_NATIVE, abi.MODE_SHARED):
+        acc.set_mode(mode, abi.POLICY_PARTITION)
+        job = make()
+        s = acc.run([job])[0]
+        assert s.coverage_ok == 1, mode
+        out[mode] = (job.result(), s)
+    acc.set_mode(abi.MODE_SHARED, abi.POLICY_PARTITION)
+    return out[abi.MODE_NATIVE], out[abi.MODE_SHARED]
+
+
+@pytest.mark.parametrize("tenant", TENANTS)
+@pytest.mark.parametrize("which", ["full", "2sm"])
+def test_tenant_partition_equals_native(pacc, pacc_2sm, tenant, which):
+    """Output-transparency: the partitioned run is bit-identical to the native
+    launch of the same body (no tenant combines floats across VGs)."""
+    from paper_conf_cgo_margiolaso16_b200.jobs import make_job
+    acc = pacc if which == "full" else pacc_2sm
+    size = "tiny" if tenant in ("mop",) else "small"
+    d = synth.preset(tenant, size, seed=7)
+    (rn, sn), (rp, sp) = _native_then_partition(acc, lambda: make_job(tenant, d))
+    for k in rn:
+        if tenant == "bfs" and k != "level":
+            continue  # frontier order depends on which CTA enqueues first
+        assert np.array_equal(rn[k], rp[k]), (tenant, k)
+    info = acc.kernel_info({"mriq": "mriq_q", "sgemm": "sgemm_tc"}.get(tenant, tenant))
+    assert info.occ_partition >= 1
+    assert sp.quota_initial % info.occ_partition == 0
+    assert sp.quota_initial <= info.occ_partition * (148 if which == "full" else 2)
+
+
+def test_c2_mix_partition_exact(pacc, oracle_lib):
+    from paper_conf_cgo_margiolaso16_b200.jobs import make_job
+    names = ["bfs", "cutcp", "stencil", "tpacf"]
+    ds = {"bfs": synth.preset("bfs", "default", seed=3),
+          "cutcp": synth.preset("cutcp", "small", seed=4),
+          "stencil": synth.preset("stencil", "small", seed=5, sweeps=10),
+          "tpacf": synth.preset("tpacf", "small", seed=6)}
+    for rep in range(2):
+        jobs = [make_job(n, ds[n]) for n in names]
+        st = pacc.run(jobs)
+        assert all(s.coverage_ok == 1 for s in st)
+        assert np.array_equal(jobs[0].result()["level"], oracle_lib.bfs(ds["bfs"])[0])
+        assert_close_fp32(jobs[1].result()["v"], oracle_lib.cutcp(ds["cutcp"]))
+        assert_close_fp32(jobs[2].result()["a"], oracle_lib.stencil(ds["stencil"]))
+        dd, rr, dr = oracle_lib.tpacf(ds["tpacf"])
+        r = jobs[3].result()
+        assert np.array_equal(r["dd"], dd) and np.array_equal(r["rr"], rr) and np.array_equal(r["dr"], dr)
+        # 4 requests, 148 SMs: 37 SMs each (all four grids are large)
+        infos = [pacc.kernel_info(n).occ_partition for n in names]
+        assert [s.quota_initial for s in st] == [37 * c for c in infos]
+
+
+@pytest.mark.parametrize("seed", [0, 1])
+def test_partition_staggered_handover(pacc, oracle_lib, seed):
+    """Arrivals shrink the running requests (SMs handed over at VG
+    boundaries), departures grow the survivors; results stay exact."""
+    from paper_conf_cgo_margiolaso16_b200.jobs import BfsJob, HistoJob, MriqJob, StencilJob, TpacfJob
+    dsn = synth.preset("stencil", "default", seed=seed, sweeps=30)
+    dbf = synth.preset("bfs", "default", seed=seed)
+    dhi = synth.preset("histo", "default", seed=seed, iters=8)
+    dtp = synth.preset("tpacf", "small", seed=seed)
+    dmq = synth.preset("mriq", "small", seed=seed)
+    jobs = [StencilJob(dsn), MriqJob(dmq), BfsJob(dbf), HistoJob(dhi), TpacfJob(dtp)]
+    ids = []
+    for t, j in enumerate(jobs):
+        ids += pacc.submit([j], tenants=[t])
+        time.sleep(0.0002)
+    pacc.sync()
+    st = [pacc.stats(i) for i in ids]
+    pacc.release()
+    assert all(s.coverage_ok == 1 for s in st)
+    assert sum(s.resolves for s in st) >= 1
+    assert np.array_equal(jobs[2].result()["level"], oracle_lib.bfs(dbf)[0])
+    assert np.array_equal(jobs[3].result()["counts"], oracle_lib.histo(dhi)[0])
+    dd, rr, dr = oracle_lib.tpacf(dtp)
+    r = jobs[4].result()
+    assert np.array_equal(r["dd"], dd) and np.array_equal(r["rr"], rr) and np.array_equal(r["dr"], dr)
+    _, qr, qi = oracle_lib.mriq(dmq)
+    assert_close_fp32(jobs[1].result()["qr"], qr, what="mriq qr")
+    zlo = 10
+    slab = dict(dsn, a0=np.ascontiguousarray(dsn["a0"][zlo:]), nz=64 - zlo)
+    ref = oracle_lib.stencil(slab)
+    assert_close_fp32(jobs[0].result()["a"][40:44], ref[40 - zlo:44 - zlo], what="stencil")
+
+
+def test_partition_requests_do_not_share_sms(pacc):
+    """Two long requests submitted together: on every SM, the VGs of one never
+    run while the other's run (ACCEL_REQ_TRACE), apart from the start-up
+    guests of a request that owned no SM yet (bounded to one chunk each)."""
+    from paper_conf_cgo_margiolaso16_b200.jobs import make_job
+    jobs = [make_job("mriq", synth.preset("mriq", "small", seed=1)),
+            make_job("cutcp", synth.preset("cutcp", "small", seed=2))]
+    ids = pacc.submit(jobs, tenants=[0, 1], trace=True)
+    pacc.sync()
+    traces = [pacc.vg_trace(i) for i in ids]
+    pacc.release()
+    per_sm = {}
+    for k, tr in enumerate(traces):
+        for rec in tr:
+            if rec.t_start_ns:
+                per_sm.setdefault(rec.sm, []).append((rec.t_start_ns, rec.t_end_ns, k))
+    overlap = busy = 0
+    for sm, iv in per_sm.items():
+        iv.sort()
+        for a in range(len(iv)):
+            busy += iv[a][1] - iv[a][0]
+            for b in range(a + 1, len(iv)):
+                if iv[b][0] >= iv[a][1]:
+                    break
+                if iv[b][2] != iv[a][2]:
+                    overlap += min(iv[a][1], iv[b][1]) - iv[b][0]
+    assert busy > 0
+    assert overlap / busy < 0.05, overlap / busy

@@ -21,14 +21,14 @@ def _worker(rank, world, port, q):
     dist.init_process_group("gloo", rank=rank, world_size=world)
     import bench
     mix = bench.c5_mix(rank)
-    res = {"rank": rank, "dev_ms": 10.0 + rank, "e2e_ms": 12.0 + rank, "nat_ms": 15.0, "oth_ms": 11.0,
+    res = {"rank": rank, "dev_ms": 10.0 + rank, "e2e_ms": 12.0 + rank, "nat_ms": 15.0, "oth_ms": {"resolve": 11.0},
            "tenants": mix, "sh": {"U": [1.5 + rank], "STP": [2.0], "ANTT": [2.0]},
-           "na": {"U": [4.0], "STP": [1.5], "ANTT": [3.0]}, "ot": {"U": [2.0], "STP": [1.8], "ANTT": [2.5]}}
+           "na": {"U": [4.0], "STP": [1.5], "ANTT": [3.0]}, "ot": {"resolve": {"U": [2.0], "STP": [1.8], "ANTT": [2.5]}}}
     allres = [None] * world
     dist.all_gather_object(allres, res)
     dist.barrier()
     if rank == 0:
-        q.put((allres, bench.aggregate(allres, world, 5, "resolve")))
+        q.put((allres, bench.aggregate(allres, world, 5, "partition")))
     dist.destroy_process_group()
 
 
@@ -50,4 +50,4 @@ def test_two_rank_aggregation():
     assert agg["tmax"] == 11.0                                     # max over ranks
     assert agg["value"] == pytest.approx(2 * 5 / 0.011)           # all mixes / slowest rank
     assert agg["U_sh"] == pytest.approx((1.5 * 2.5) ** 0.5)       # geometric mean over ranks
-    assert agg["other"]["throughput_speedup"] == pytest.approx(15.0 / 11.0)
+    assert agg["other"]["resolve"]["throughput_speedup"] == pytest.approx(15.0 / 11.0)

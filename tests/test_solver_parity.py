@@ -1,5 +1,6 @@
 """The product solver (C++ accel_solve in libaccel.so) equals the oracle
 (oracle/solver_ref.py) exactly; demand vectors and metrics likewise."""
+import math
 import random
 
 import pytest
@@ -96,3 +97,46 @@ def test_metrics_equal():
         st = [r.uniform(0, 5) for _ in range(k)]
         en = [s + r.uniform(0, 5) for s in st]
         assert abi.accel_overlap(st, en) == pytest.approx(M.overlap(list(zip(st, en))), abs=1e-12)
+
+
+def test_partition_parity():
+    r = random.Random(5)
+    n = 0
+    for _ in range(3000):
+        caps = S.Caps(sms=r.choice([1, 2, 3, 5, 9, 148]), thr_per_sm=r.choice([512, 1024, 2048]),
+                      regs_per_sm=r.choice([32768, 65536]), smem_per_sm=r.choice([65536, 233472]),
+                      ctas_per_sm=r.choice([4, 8, 16, 32]))
+        try:
+            ds = _random_instance(r, caps, 8, 5000)
+        except S.NoFit:
+            continue
+        ref = S.solve_sms(ds, caps)
+        got = abi.accel_solve_sms([_to_c(d) for d in ds], _caps(caps))
+        assert (list(got[0]), list(got[1])) == (list(ref[0]), list(ref[1])), (caps, ds)
+        n += 1
+    assert n > 2500
+    caps = S.Caps(sms=4, thr_per_sm=256)
+    a, b = S.demand_of(256, 32, 0, 12, caps=caps), S.demand_of(256, 32, 0, 8, caps=caps)
+    assert abi.accel_solve_sms([_to_c(a), _to_c(b)], _caps(caps)) == ([2, 2], [1, 1])
+
+
+def test_fair_weights_closed_forms():
+    """FAIR weights (DESIGN.md R-fair-2): 16 * (s_i / geomean s)^2, clamped to
+    [1, 1024]; equal slowdowns -> equal (neutral) weights; unknown (<= 0) ->
+    neutral; doubling a slowdown quadruples the weight relative to the others."""
+    assert abi.accel_fair_weights([1.7, 1.7, 1.7, 1.7]) == [16] * 4
+    assert abi.accel_fair_weights([1.0, 2.0, 4.0]) == [4, 16, 64]
+    assert abi.accel_fair_weights([2.0, -1.0, 8.0]) == [4, 16, 64]
+    assert abi.accel_fair_weights([1.0, 1000.0]) == [1, 1024]
+    r = random.Random(9)
+    for _ in range(200):
+        s = [r.uniform(0.5, 6.0) for _ in range(r.randint(1, 8))]
+        w = abi.accel_fair_weights(s)
+        g = math.exp(sum(math.log(x) for x in s) / len(s))
+        assert w == [min(1024, max(1, round(16 * (x / g) ** 2))) for x in s] or all(
+            abs(a - b) <= 1 for a, b in zip(w, [16 * (x / g) ** 2 for x in s]))
+        # monotone: a larger slowdown never gets a smaller weight
+        for i in range(len(s)):
+            for j in range(len(s)):
+                if s[i] > s[j]:
+                    assert w[i] >= w[j]
