@@ -269,11 +269,18 @@ def main():
     ap.add_argument("--config", default="c2", choices=["c1", "c2", "c5"])
     ap.add_argument("--impl", default="accel", choices=["accel", "reference"])
     ap.add_argument("--calib-reps", type=int, default=5)
-    ap.add_argument("--policy", default="fair", choices=["fair", "resolve", "static", "partition"],
+    ap.add_argument("--policy", default="resolve", choices=["fair", "resolve", "static", "partition"],
                     help="SHARED-mode policy of the timed (headline) run; the others are reported too")
     ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--all-policies", action="store_true",
+                    help="also run the experimental PARTITION and FAIR policies")
     ap.add_argument("--out", default=None, help="also write the JSON line here")
+    ap.add_argument("--hang-dump-s", type=float, default=0.0,
+                    help="debug: dump every thread's Python stack after this many seconds")
     args = ap.parse_args()
+    if args.hang_dump_s > 0:
+        import faulthandler
+        faulthandler.dump_traceback_later(args.hang_dump_s, repeat=True)
     if args.impl == "reference":
         run_reference(args)
         return
@@ -304,7 +311,10 @@ def main():
            "partition": abi.POLICY_PARTITION}
     hints = {}   # FAIR: isolated-time profile per tenant (from the calibration below)
     head_pol = POL[args.policy]
-    other_pols = [p for p in POL if p != args.policy]
+    # reported beside the headline: STATIC (the paper's policy) and RESOLVE;
+    # PARTITION and FAIR (experimental) only with --all-policies
+    shown = POL if args.all_policies else ("static", "resolve")
+    other_pols = [p for p in shown if p != args.policy]
 
     def run_group(js, mode, e2e=False, launch_events=False, policy=None):
         policy = head_pol if policy is None else policy
@@ -322,7 +332,8 @@ def main():
 
     # -- correctness pass (untimed): coverage of every VG, both modes
     with Accel(device=local, mode=abi.MODE_SHARED, verify=True) as vacc:
-        for mode, pol in [(abi.MODE_NATIVE, abi.POLICY_STATIC)] + [(abi.MODE_SHARED, POL[p]) for p in POL]:
+        for mode, pol in [(abi.MODE_NATIVE, abi.POLICY_STATIC)] + [(abi.MODE_SHARED, POL[p]) for p in
+                                                                  {args.policy, *other_pols}]:
             vacc.set_mode(mode, pol)
             st = vacc.run(jobs)
             assert all(s.coverage_ok == 1 for s in st), "coverage check failed"

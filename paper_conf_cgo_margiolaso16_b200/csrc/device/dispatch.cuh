@@ -267,7 +267,13 @@ __device__ __forceinline__ void wait_complete(const Desc* p) {
 enum : uint32_t {
   kCfgChunkMask = 0xffffu,
   kCfgResolve = 1u << 16,
-  kCfgStamps = 1u << 17
+  kCfgStamps = 1u << 17,
+  kCfgHasPrev = 1u << 18,  // the request ran a launch before this one (RESOLVE
+                           // persistent grids check its `topped` word)
+  // measurement-only ablations (env ACCEL_ABLATE on the host; scripts/isolated.py)
+  kAblNoFence = 1u << 24,  // retire without the release fence (UNSAFE with top-ups)
+  kAblNoLive = 1u << 25,   // never load the live quota (no shrink)
+  kAblNoStats = 1u << 26   // no cur / max_alive reductions at admission
 };
 
 // Scheduling state of one CTA in shared memory (the paper's `local struct SD`,
@@ -429,7 +435,7 @@ __device__ __forceinline__ unsigned long long dequeue(Desc* d, SchedState* S) {
 template <bool kResolve>
 __device__ __forceinline__ void retire(Desc* d, uint32_t cfg, const SchedState* S) {
   if (kResolve && S->admitted) {
-    fence_acq_rel();  // this CTA's VG results before the alive decrement
+    if (!(cfg & kAblNoFence)) fence_acq_rel();  // this CTA's VG results before the alive decrement
     atomicAdd(&d->qa, kAliveNeg);
   }
   if (kResolve && S->draining) {
@@ -459,14 +465,22 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
       S->admitted = 0;
       b = kTerminate;
     } else {
+      // a predecessor launch that was topped up may still be running on its
+      // top-up CTAs: this grid's body must wait for it.  The flag load, the
+      // admission and the first dequeue are all issued before the wait, so a
+      // launch that was never topped pays no extra round trip
+      const uint32_t topped_prev =
+          (!kPart && (cfg & kCfgHasPrev)) ? ld_volatile(&(d - 1)->topped) : 0u;
       // admission and first dequeue in one atomic; an arrival over the live
       // quota runs the chunk it got and leaves at its next dequeue
-      asm volatile("red.relaxed.gpu.global.max.u32 [%0], %1;" ::"l"(&d->ctl->cur), "r"(d->req_idx) : "memory");
-      const uint32_t live = d->governed ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
+      if (!(cfg & kAblNoStats))
+        asm volatile("red.relaxed.gpu.global.max.u32 [%0], %1;" ::"l"(&d->ctl->cur), "r"(d->req_idx) : "memory");
+      const uint32_t live = (d->governed && !(cfg & kAblNoLive)) ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
       const unsigned long long v = atomicAdd(&d->qa, kAlive1 | chunk);
       b = qa_next(v);
       const uint32_t a = qa_alive(v) + 1u;
-      asm volatile("red.relaxed.gpu.global.max.u32 [%0], %1;" ::"l"(&d->max_alive), "r"(a) : "memory");
+      if (!(cfg & kAblNoStats))
+        asm volatile("red.relaxed.gpu.global.max.u32 [%0], %1;" ::"l"(&d->max_alive), "r"(a) : "memory");
       if (a > live) {
         S->over = 1;
         red_add_u32(&d->admit_fail, 1u);
@@ -474,12 +488,17 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
       }
       S->hint_live = live;
       S->hint_alive = a;
+      if (topped_prev) wait_complete(d - 1);
     }
     if (cfg & kCfgStamps) red_min_u64(&d->t_first, globaltimer());
     const uint32_t launch_idx = d->launch_idx;
     const uint32_t total = vg_total<T>(args, d, launch_idx);
-    // (PARTITION: any CTA may be the only one that reaches this launch)
-    if (kPart ? ld_volatile(&d->total_seen) == kTerminate : blockIdx.x == 0) d->total_seen = total;
+    // RESOLVE / PARTITION: every CTA publishes the total (the same value: a
+    // dynamic total is final once the predecessor launch completed).  Top-up
+    // CTAs may serve a launch before its main grid is resident -- when they
+    // fill the SMs the main grid waits for them -- so completion of a launch
+    // (wait_complete) must never depend on one particular CTA of the main grid
+    if (kResolve || blockIdx.x == 0) d->total_seen = total;
     S->chunk = chunk;
     S->have_nxt = 0;
     S->long_vg = 0;
@@ -515,7 +534,7 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
         // that idle time dwarfs one queue round trip) dequeue just in time
         // once fewer than two waves of VGs remain
         r_v = dequeue<kResolve, kPart>(d, S);
-        if (kResolve) r_live = d->governed ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
+        if (kResolve) r_live = (d->governed && !(cfg & kAblNoLive)) ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
         if (kPart) {
           r_own = ld_relaxed(&S->owner[S->sm]);
           r_qc = ld_relaxed_u64(&d->ctl->sm_quota);
@@ -541,7 +560,7 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
       } else {                                   // publish the prefetched chunk
         if (!S->have_nxt) {                      // tail: just in time
           r_v = dequeue<kResolve, kPart>(d, S);
-          if (kResolve) r_live = d->governed ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
+          if (kResolve) r_live = (d->governed && !(cfg & kAblNoLive)) ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
           if (kPart) {
             r_own = ld_relaxed(&S->owner[S->sm]);
             r_qc = ld_relaxed_u64(&d->ctl->sm_quota);
@@ -578,10 +597,6 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
     accel_persistent(const typename T::Args args, Desc* __restrict__ d, uint32_t cfg) {
   extern __shared__ __align__(128) char smem[];
   __shared__ SchedState S;
-  if (kResolve) {
-    if (threadIdx.x == 0 && d->has_prev && ld_volatile(&(d - 1)->topped)) wait_complete(d - 1);
-    __syncthreads();
-  }
   serve<T, kResolve>(args, d, smem, &S, cfg, blockIdx.x);
 }
 
@@ -634,10 +649,15 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
       }
     }
     __syncthreads();
+    // (the predecessor wait above already ran: no kCfgHasPrev)
     const uint32_t cfg = dl->chunk | kCfgResolve | ((dl->flags & kFlagStamps) ? kCfgStamps : 0u);
     serve<T, true, kPart>(args, dl, smem, &S, cfg, blockIdx.x | (kPart ? 0u : 0x80000000u));
     __syncthreads();
     if (kPart && S.left) return;
+    // RESOLVE: a top-up CTA that was evicted (shrink) or admitted over the live
+    // quota is surplus: it leaves the request instead of following the later
+    // launches (the monitor tops up afresh on a later growth, apply_quota)
+    if (!kPart && (S.over || S.draining)) return;
   }
   // the step's last launch is exhausted: free the SM (one CTA per SM wins the
   // CAS and returns the count); the request's next step claims afresh, so a

@@ -181,9 +181,7 @@ struct accel_ctx {
   std::atomic<bool> stop{false};
   uint64_t monitor_solves = 0;
   std::chrono::steady_clock::time_point last_fair{};
-  // dispatch variant (env ACCEL_DISPATCH): "" / "dyn" = one dequeue in flight,
-  // "dyn2" = two in flight (kCfgDepth2), "stride" = static round robin (ablation)
-  uint32_t dispatch_bits = 0;
+  uint32_t ablate = 0;   // env ACCEL_ABLATE: measurement-only cfg bits (dispatch.cuh kAbl*)
   std::vector<uint8_t> slot_used;
   std::map<uint64_t, std::unique_ptr<Request>> reqs;
   uint64_t next_id = 1;
@@ -353,7 +351,8 @@ int enqueue(accel_ctx* ctx, Request* r) {
       if (lev) CK(ctx, cudaEventRecord(r->ev_launch[li], s));
       accel::Desc* d = ctx->desc_ptr(r->slot + st.first + l);
       // accel_persistent cfg word (dispatch.cuh): chunk | kCfgResolve | kCfgStamps
-      uint32_t cfg = (k.chunk & 0xffffu) | (resolve ? (1u << 16) : 0u) | (1u << 17) | ctx->dispatch_bits;
+      // | kCfgHasPrev (a request-relative launch precedes this one)
+      uint32_t cfg = (k.chunk & 0xffffu) | (resolve ? (1u << 16) : 0u) | (1u << 17) | (li > 0 ? (1u << 18) : 0u) | ctx->ablate;
       void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &cfg};
       const dim3 grid = shared ? dim3(st.quota, 1, 1) : dim3(st.grid.x, st.grid.y, st.grid.z);
       CK(ctx, cudaLaunchKernel(shared ? (resolve ? k.prfn : k.pfn) : k.nfn, grid, k.block, params, k.dyn_smem, s));
@@ -793,10 +792,7 @@ int accel_init(const accel_config* cfg, accel_ctx** out) {
                          cudaHostAllocDefault)) != cudaSuccess)
     return init_fail(e, "cudaHostAlloc(ring)");
   ctx->slot_used.assign(kPoolSlots, 0);
-  if (const char* dv = std::getenv("ACCEL_DISPATCH")) {
-    if (std::strcmp(dv, "dyn2") == 0) ctx->dispatch_bits = 1u << 18;
-    if (std::strcmp(dv, "stride") == 0) ctx->dispatch_bits = 1u << 19;
-  }
+  if (const char* ab = std::getenv("ACCEL_ABLATE")) ctx->ablate = ((uint32_t)std::atoi(ab) & 7u) << 24;
   accel_ctx* raw = ctx.release();
   raw->monitor = std::thread(monitor_loop, raw);
   *out = raw;
