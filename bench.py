@@ -285,6 +285,9 @@ def main():
         run_reference(args)
         return
 
+    # a stalled request turns into an error with a device-state dump
+    # (accel_sync watchdog) instead of a hung bench
+    os.environ.setdefault("ACCEL_SYNC_TIMEOUT_S", "120")
     import torch
     import torch.distributed as dist
 
@@ -314,6 +317,8 @@ def main():
     # reported beside the headline: STATIC (the paper's policy) and RESOLVE;
     # PARTITION and FAIR (experimental) only with --all-policies
     shown = POL if args.all_policies else ("static", "resolve")
+    if not os.environ.get("ACCEL_EXPERIMENTAL_PARTITION"):
+        shown = [p for p in shown if p != "partition"]
     other_pols = [p for p in shown if p != args.policy]
 
     def run_group(js, mode, e2e=False, launch_events=False, policy=None):

@@ -56,7 +56,10 @@ typedef enum { ACCEL_MODE_NATIVE = 0, ACCEL_MODE_SHARED = 1 } accel_mode;
  * its persistent CTAs claim SMs on the device (a per-SM owner word) and run
  * c_i per SM, padded in shared memory so that no other kernel's CTA fits
  * beside them; re-solved on every arrival and departure (an SM is handed over
- * at a VG boundary).  One persistent grid serves all launches of a step. */
+ * at a VG boundary).  One persistent grid serves all launches of a step.
+ * EXPERIMENTAL, disabled: accel_init / accel_set_mode return ACCEL_EINVAL
+ * for it unless the environment variable ACCEL_EXPERIMENTAL_PARTITION is set
+ * (it halved C2 throughput and one GPU test hung intermittently). */
 /* FAIR: RESOLVE whose weights follow the requests' measured slowdowns: the
  * monitor reads each running request's completed VGs every few hundred
  * microseconds, estimates its slowdown so far against its isolated time
@@ -209,12 +212,16 @@ typedef struct {
 /* Submit one request (solver run over the active set incl. this one).
  * Non-blocking; *request_id identifies it for sync/stats. */
 int accel_submit(accel_ctx *ctx, const accel_request *r, uint64_t *request_id);
-/* Submit n requests that arrive together: ONE solve over all of them, then
- * enqueue in array order (the mix order decides the FCFS winner in NATIVE
- * mode). request_ids[n] out. */
+/* Submit n requests that arrive together: ONE solve over all of them.
+ * NATIVE mode enqueues them in array order (the mix order decides the FCFS
+ * winner); SHARED mode enqueues the largest per-CTA
+ * footprint first (DESIGN.md R-place-1).  request_ids[n] out, in array order
+ * (ids are the arrival order of later re-solves). */
 int accel_submit_group(accel_ctx *ctx, uint32_t n, const accel_request *rs, uint64_t *request_ids);
 /* Block until request_id (or every request: ACCEL_ALL) completed.  In verify
- * mode also checks coverage -> ACCEL_ECOVERAGE. */
+ * mode also checks coverage -> ACCEL_ECOVERAGE.  Debug: with the environment
+ * variable ACCEL_SYNC_TIMEOUT_S=<seconds> set, a wait longer than that prints
+ * every unfinished launch's device state to stderr and returns ACCEL_ESTATE. */
 int accel_sync(accel_ctx *ctx, uint64_t request_id);
 /* Record the time origin for accel_req_stats.arrival_ms / done_ms on every
  * tenant stream (call between mixes, when idle). */

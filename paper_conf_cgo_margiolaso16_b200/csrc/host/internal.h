@@ -43,6 +43,6 @@ cudaError_t launch_desc_init(const InitParams& p, uint32_t n_desc, cudaStream_t 
 // PARTITION: then release the SMs the request still owns (nsm owner words).
 cudaError_t launch_join(const Desc* last, uint32_t nsm, cudaStream_t s);
 constexpr size_t kDescBytes = 384;
-constexpr size_t kCtlBytes = 32;
+constexpr size_t kCtlBytes = 256;
 
 }  // namespace accel

@@ -605,7 +605,7 @@ bool fair_weights(accel_ctx* ctx) {
   ctx->ring_pos += (uint32_t)rs.size();
   if (ctx->ring_pos % kRing < rs.size()) return false;  // wrap: skip this round
   for (size_t i = 0; i < rs.size(); ++i)
-    if (ctx->cuda(cudaMemcpyAsync(h + i, ctx->ctl_pool + (size_t)rs[i]->slot * kCtlBytes + 16 /* done_vgs */,
+    if (ctx->cuda(cudaMemcpyAsync(h + i, ctx->ctl_pool + (size_t)rs[i]->slot * kCtlBytes + 132 /* Ctl::done_vgs */,
                                   sizeof(uint32_t), cudaMemcpyDeviceToHost, ctx->ctl),
                   "cudaMemcpyAsync(progress)"))
       return false;
@@ -706,11 +706,34 @@ int submit_locked(accel_ctx* ctx, uint32_t n, const accel_request* rs, uint64_t*
     if (r->cov_elems) CK(ctx, cudaMalloc(&r->cov, r->cov_elems * sizeof(uint32_t)));
     if (r->trace_elems) CK(ctx, cudaMalloc(&r->trace, r->trace_elems * sizeof(accel_vg_record)));
   }
-  for (uint32_t i = 0; i < n; ++i) {
+  // SHARED: requests that arrive together are enqueued largest per-CTA
+  // footprint first (dominant share of one SM, DESIGN.md R-place-1).  The
+  // block scheduler places each grid breadth-first over the SMs with room
+  // left; the solver's packing (F) puts ceil(n_i / S) CTAs of every kernel
+  // on an SM, which a big-CTA kernel (tensor-core sgemm: one CTA per SM by
+  // shared memory) only gets if it is placed before small CTAs fragment the
+  // SMs -- otherwise it waits for a whole co-runner to finish.  NATIVE keeps
+  // the mix order (its FCFS winner is the point of the baseline).
+  std::vector<uint32_t> ord(n);
+  for (uint32_t i = 0; i < n; ++i) ord[i] = i;
+  if (ctx->cfg.mode == ACCEL_MODE_SHARED) {
+    std::vector<double> fp(n, 0.0);
+    for (uint32_t i = 0; i < n; ++i) {
+      accel_demand d{};
+      if (demand_for(ctx, fresh[i]->steps[fresh[i]->main_step], 1, &d) == ACCEL_OK)
+        fp[i] = std::max({(double)d.thr / ctx->caps.thr_per_sm, (double)d.regs / ctx->caps.regs_per_sm,
+                          (double)d.smem / ctx->caps.smem_per_sm, (double)d.cta / ctx->caps.ctas_per_sm});
+    }
+    std::stable_sort(ord.begin(), ord.end(), [&](uint32_t a, uint32_t b) { return fp[a] > fp[b]; });
+  }
+  // ids (= arrival order for later re-solves) follow the array order
+  const uint64_t base = ctx->next_id;
+  ctx->next_id += n;
+  for (uint32_t i : ord) {
     Request* r = fresh[i].get();
     int rc = enqueue(ctx, r);
     if (rc) return rc;
-    r->id = ctx->next_id++;
+    r->id = base + i;
     ids[i] = r->id;
     ctx->reqs[r->id] = std::move(fresh[i]);
   }
@@ -752,12 +775,21 @@ const char* accel_last_error(const accel_ctx* ctx) {
   return ctx ? ctx->err.c_str() : g_init_error.c_str();
 }
 
+// PARTITION is experimental and off unless ACCEL_EXPERIMENTAL_PARTITION is
+// set: it lost half the native throughput on C2 and one of its single-tenant
+// GPU tests hung intermittently
+bool policy_enabled(int32_t policy) {
+  if (policy == ACCEL_POLICY_STATIC || policy == ACCEL_POLICY_RESOLVE || policy == ACCEL_POLICY_FAIR) return true;
+  return policy == ACCEL_POLICY_PARTITION && std::getenv("ACCEL_EXPERIMENTAL_PARTITION") != nullptr;
+}
+
 int accel_init(const accel_config* cfg, accel_ctx** out) {
   if (!cfg || !out) return ACCEL_EINVAL;
   if (cfg->mode != ACCEL_MODE_NATIVE && cfg->mode != ACCEL_MODE_SHARED) return ACCEL_EINVAL;
-  if (cfg->policy != ACCEL_POLICY_STATIC && cfg->policy != ACCEL_POLICY_RESOLVE &&
-      cfg->policy != ACCEL_POLICY_PARTITION && cfg->policy != ACCEL_POLICY_FAIR)
+  if (!policy_enabled(cfg->policy)) {
+    g_init_error = "bad or disabled policy (PARTITION needs ACCEL_EXPERIMENTAL_PARTITION=1)";
     return ACCEL_EINVAL;
+  }
   auto ctx = std::make_unique<accel_ctx>();
   ctx->cfg = *cfg;
   auto init_fail = [&](cudaError_t e, const char* what) {
@@ -830,9 +862,8 @@ int accel_set_mode(accel_ctx* ctx, int32_t mode, int32_t policy) {
   std::lock_guard<std::mutex> g(ctx->mu);
   if (ctx->poisoned) return ACCEL_ESTATE;
   if (mode != ACCEL_MODE_NATIVE && mode != ACCEL_MODE_SHARED) return ctx->fail(ACCEL_EINVAL, "bad mode");
-  if (policy != ACCEL_POLICY_STATIC && policy != ACCEL_POLICY_RESOLVE && policy != ACCEL_POLICY_PARTITION &&
-      policy != ACCEL_POLICY_FAIR)
-    return ctx->fail(ACCEL_EINVAL, "bad policy");
+  if (!policy_enabled(policy))
+    return ctx->fail(ACCEL_EINVAL, "bad or disabled policy (PARTITION needs ACCEL_EXPERIMENTAL_PARTITION=1)");
   for (auto& kv : ctx->reqs) {
     int rc = refresh_done(ctx, kv.second.get());
     if (rc) return rc;
@@ -950,6 +981,45 @@ int accel_submit(accel_ctx* ctx, const accel_request* r, uint64_t* id) {
   return accel_submit_group(ctx, 1, r, id);
 }
 
+// Debug (ACCEL_SYNC_TIMEOUT_S): print every unfinished request's launches as
+// the device sees them (descriptors copied on a fresh stream by the copy
+// engine, which works while kernels spin).
+void dump_stuck(accel_ctx* ctx, const std::vector<uint64_t>& ids) {
+  cudaStream_t st;
+  if (cudaStreamCreateWithFlags(&st, cudaStreamNonBlocking) != cudaSuccess) return;
+  for (uint64_t id : ids) {
+    auto it = ctx->reqs.find(id);
+    if (it == ctx->reqs.end()) continue;
+    Request* r = it->second.get();
+    if (cudaEventQuery(r->ev_done) == cudaSuccess) continue;
+    std::vector<unsigned char> h((size_t)r->n_desc * kDescBytes);
+    uint32_t ctl[2] = {0, 0};
+    void* hp = nullptr;
+    if (cudaHostAlloc(&hp, h.size() + 256, cudaHostAllocDefault) != cudaSuccess) break;
+    cudaMemcpyAsync(hp, ctx->desc_ptr(r->slot), h.size(), cudaMemcpyDeviceToHost, st);
+    cudaMemcpyAsync((char*)hp + h.size(), ctx->ctl_pool + (size_t)r->slot * kCtlBytes, 256, cudaMemcpyDeviceToHost, st);
+    const auto t0 = std::chrono::steady_clock::now();
+    while (cudaStreamQuery(st) == cudaErrorNotReady &&
+           std::chrono::steady_clock::now() - t0 < std::chrono::seconds(5))
+      std::this_thread::sleep_for(std::chrono::milliseconds(1));
+    std::memcpy(h.data(), hp, h.size());
+    std::memcpy(ctl, (char*)hp + h.size(), sizeof(uint32_t));
+    std::memcpy(ctl + 1, (char*)hp + h.size() + 128, sizeof(uint32_t));
+    cudaFreeHost(hp);
+    std::fprintf(stderr, "[accel] STUCK req %llu tenant %d live(host) %u provisioned %u topups %zu | ctl live %u cur %u\n",
+                 (unsigned long long)id, r->tenant, r->live, r->provisioned, r->ev_topups.size(), ctl[0], ctl[1]);
+    for (uint32_t l = 0; l < r->n_desc; ++l) {
+      const DescHost* d = reinterpret_cast<const DescHost*>(h.data() + (size_t)l * kDescBytes);
+      const uint32_t next = (uint32_t)d->qa, alive = (uint32_t)(d->qa >> 32);
+      if (d->total_seen != 0xffffffffu && next >= d->total_seen && alive == 0 && d->draining == 0) continue;
+      std::fprintf(stderr, "[accel]   launch %u: total %u seen %u next %u alive %u draining %u topped %u started %u "
+                           "refused %u evicted %u\n", l, d->total, d->total_seen, next, alive, d->draining, d->topped,
+                   d->ctas_started, d->admit_fail, d->evicted);
+    }
+  }
+  cudaStreamDestroy(st);
+}
+
 int accel_sync(accel_ctx* ctx, uint64_t request_id) {
   if (!ctx) return ACCEL_EINVAL;
   std::vector<uint64_t> ids;
@@ -979,8 +1049,22 @@ int accel_sync(accel_ctx* ctx, uint64_t request_id) {
       }
     }
     if (wait.empty()) break;
+    static const double watchdog_s = std::getenv("ACCEL_SYNC_TIMEOUT_S") ? std::atof(std::getenv("ACCEL_SYNC_TIMEOUT_S")) : 0.0;
+    const auto t0 = std::chrono::steady_clock::now();
     for (cudaEvent_t ev : wait) {
-      cudaError_t e = cudaEventSynchronize(ev);
+      cudaError_t e;
+      if (watchdog_s > 0.0) {   // debug: poll, and on timeout dump the launches' device state
+        while ((e = cudaEventQuery(ev)) == cudaErrorNotReady) {
+          if (std::chrono::duration<double>(std::chrono::steady_clock::now() - t0).count() > watchdog_s) {
+            std::lock_guard<std::mutex> g(ctx->mu);
+            dump_stuck(ctx, ids);
+            return ctx->fail(ACCEL_ESTATE, "accel_sync watchdog: requests did not complete (state dumped to stderr)");
+          }
+          std::this_thread::sleep_for(std::chrono::microseconds(200));
+        }
+      } else {
+        e = cudaEventSynchronize(ev);
+      }
       if (e != cudaSuccess) {
         std::lock_guard<std::mutex> g(ctx->mu);
         return ctx->cuda(e, "cudaEventSynchronize");

@@ -10,7 +10,13 @@ import pytest
 import synth
 from tests.gpu_util import assert_close_fp32
 
-pytestmark = pytest.mark.gpu
+import os
+
+# PARTITION is experimental and disabled in the library unless
+# ACCEL_EXPERIMENTAL_PARTITION is set (an intermittent hang)
+pytestmark = [pytest.mark.gpu,
+              pytest.mark.skipif(not os.environ.get("ACCEL_EXPERIMENTAL_PARTITION"),
+                                 reason="PARTITION policy disabled (ACCEL_EXPERIMENTAL_PARTITION unset)")]
 
 TENANTS = ["mop", "stencil", "histo", "bfs", "cutcp", "tpacf", "spmv", "sgemm", "mriq"]
 
@@ -143,9 +149,9 @@ def test_partition_requests_do_not_share_sms(pacc):
     pacc.release()
     per_sm = {}
     for k, tr in enumerate(traces):
-        for rec in tr:
-            if rec.t_start_ns:
-                per_sm.setdefault(rec.sm, []).append((rec.t_start_ns, rec.t_end_ns, k))
+        for rec in tr:   # numpy structured records (abi.accel_vg_trace)
+            if rec["t_start_ns"]:
+                per_sm.setdefault(int(rec["sm"]), []).append((int(rec["t_start_ns"]), int(rec["t_end_ns"]), k))
     overlap = busy = 0
     for sm, iv in per_sm.items():
         iv.sort()
