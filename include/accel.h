@@ -286,6 +286,12 @@ int accel_demand_of(const accel_caps *caps, uint32_t block_threads, uint32_t reg
 /* The share solver of PAPER.md §3 (closed form + per-SM feasibility + greedy),
  * k requests in arrival order -> quota_out[k]. */
 int accel_solve(const accel_caps *caps, const accel_demand *d, int32_t k, uint32_t *quota_out);
+/* Placement order of k requests (DESIGN.md R-place-1): order_out[k] = request
+ * indices, largest per-CTA footprint (max over threads, registers, shared
+ * memory, CTA slots of the share of ONE SM) first, ties in arrival order.
+ * SHARED mode enqueues a group's grids in this order and the solver's
+ * feasibility model F places them in it.  ACCEL_ENOFIT for an invalid demand. */
+int accel_placement_order(const accel_caps *caps, const accel_demand *d, int32_t k, int32_t *order_out);
 /* SM-granular variant (ACCEL_POLICY_PARTITION; DESIGN.md R-part-1..4): the
  * same closed form + class-symmetric greedy with whole SMs as the one device
  * total.  sms_out[k] = SMs per request (sum <= caps->sms, each <= ceil(G/c));

@@ -23,6 +23,14 @@ Readings (DESIGN.md):
               after adding 1 KiB reserved (cuda_occupancy.h).
   R-solver-3  The closed form runs on device totals; a per-SM feasibility
               model F (below) then checks that the quotas actually pack.
+              F simulates the placement the library causes (R-place-1):
+              kernels in placement order (largest per-CTA footprint first,
+              ties by arrival), each kernel's CTAs dealt round-robin over the
+              SMs, skipping SMs where the CTA does not fit, from a pointer
+              that carries over between kernels -- the B200 block scheduler's
+              breadth-first fill.  (The first version dealt ceil/floor counts
+              on rotating offsets regardless of room: it claimed that 127
+              small CTAs occupy 127 SMs and gave a one-CTA-per-SM GEMM 21 SMs.)
   R-solver-4  A quota never exceeds the request's virtual-group count G_i;
               a request with G_i = 0 gets 0.
   R-solver-5  Requests with identical (demand, G, weight) form a class; the
@@ -141,49 +149,73 @@ def closed_form(ds: Sequence[Demand], caps: Caps = Caps()) -> list[int]:
     return out
 
 
+def footprint(d: Demand, caps: Caps = Caps()) -> Fraction:
+    """Per-CTA footprint: the largest share of ONE SM's resources a CTA takes."""
+    return max(Fraction(d.thr, caps.thr_per_sm), Fraction(d.regs, caps.regs_per_sm),
+               Fraction(d.smem, caps.smem_per_sm), Fraction(d.cta, caps.ctas_per_sm))
+
+
+def placement_order(ds: Sequence[Demand], caps: Caps = Caps()) -> list[int]:
+    """R-place-1: request indices, largest per-CTA footprint first, ties in
+    arrival order (the order the library enqueues a group's grids in)."""
+    return sorted(range(len(ds)), key=lambda i: (-footprint(ds[i], caps), i))
+
+
 def feasible(ds: Sequence[Demand], n: Sequence[int], caps: Caps = Caps()) -> bool:
     """Step 3: per-SM feasibility F(n) (R-solver-3).
 
-    Kernel i places floor(n_i/S) CTAs on every SM plus one more on n_i mod S
-    SMs, starting where kernel i-1's remainder ended (rotating offset).  On
-    every SM the thread, CTA-slot and shared-memory sums must fit, and the
-    warps must pack into the sub-partitions: each CTA (kernels in order) puts
-    its warps round-robin starting at the least-loaded SMSP (lowest index on
-    ties), and no SMSP may exceed regs_per_sm/4.
+    Kernels in placement order; kernel i's n_i CTAs are dealt round-robin over
+    the SMs from a pointer p (carried over between kernels, starting at SM 0),
+    each CTA going to the next SM where it fits: thread, CTA-slot and
+    shared-memory sums within the SM's limits, and its warps packed into the
+    sub-partitions -- round-robin from the least-loaded SMSP (lowest index on
+    ties), no SMSP above regs_per_sm/4.  F fails when a CTA fits on no SM.
+    Dealt in rounds: every SM that fits at the start of a round takes one CTA
+    (an SM is revisited only after a full cycle), the last round the first
+    SMs from p.
     """
     S = caps.sms
-    per_sm_count = [[0] * len(ds) for _ in range(S)]
-    off = 0
-    for i, d in enumerate(ds):
-        q, r = divmod(n[i], S)
-        for sm in range(S):
-            per_sm_count[sm][i] = q
-        for j in range(r):
-            per_sm_count[(off + j) % S][i] += 1
-        off = (off + r) % S
-    checked: set = set()   # SMs holding the same CTA counts give the same answer
-    for sm in range(S):
-        counts = tuple(per_sm_count[sm])
-        if counts in checked:
-            continue
-        checked.add(counts)
-        thr = cta = smem = 0
-        smsp = [0] * caps.smsp_per_sm
-        for i, d in enumerate(ds):
-            c = counts[i]
-            if c == 0:
-                continue
-            thr += c * d.thr
-            cta += c * d.cta
-            smem += c * d.smem
-            for _ in range(c):
-                start = min(range(caps.smsp_per_sm), key=lambda s: (smsp[s], s))
-                for w in range(d.warps):
-                    smsp[(start + w) % caps.smsp_per_sm] += d.rpw
-        if thr > caps.thr_per_sm or cta > caps.ctas_per_sm or smem > caps.smem_per_sm:
-            return False
-        if max(smsp) > caps.regs_per_smsp:
-            return False
+    P = caps.smsp_per_sm
+    # per-SM state (threads, CTA slots, shared memory, registers per SMSP);
+    # SMs in the same state answer alike, so the step is memoised per state
+    st = [(0, 0, 0, (0,) * P)] * S
+    memo: dict = {}
+
+    def place(state, d: Demand):
+        """The SM state after adding one CTA of d, or None if it does not fit."""
+        key = (state, d.thr, d.cta, d.smem, d.warps, d.rpw)
+        if key in memo:
+            return memo[key]
+        t, c, m, sp = state
+        out = None
+        if t + d.thr <= caps.thr_per_sm and c + d.cta <= caps.ctas_per_sm and m + d.smem <= caps.smem_per_sm:
+            start = min(range(P), key=lambda s: (sp[s], s))
+            nsp = list(sp)
+            for w in range(d.warps):
+                nsp[(start + w) % P] += d.rpw
+            if max(nsp) <= caps.regs_per_smsp:
+                out = (t + d.thr, c + d.cta, m + d.smem, tuple(nsp))
+        memo[key] = out
+        return out
+
+    p = 0
+    for i in placement_order(ds, caps):
+        d, left = ds[i], n[i]
+        while left > 0:
+            fit = []
+            for j in range(S):
+                sm = (p + j) % S
+                nxt = place(st[sm], d)
+                if nxt is not None:
+                    fit.append((sm, nxt))
+                    if len(fit) == left:
+                        break
+            if not fit:
+                return False
+            for sm, nxt in fit:
+                st[sm] = nxt
+            left -= len(fit)
+            p = (fit[-1][0] + 1) % S
     return True
 
 

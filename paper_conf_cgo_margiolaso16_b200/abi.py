@@ -163,7 +163,7 @@ EXPORTS = [
     "accel_init", "accel_finalize", "accel_set_mode", "accel_last_error", "accel_builtin_kernel",
     "accel_builtin_count", "accel_builtin_name", "accel_kernel_register", "accel_kernel_info_get",
     "accel_submit", "accel_submit_group", "accel_sync", "accel_epoch", "accel_stats", "accel_release",
-    "accel_tenant_stream", "accel_launch_times", "accel_launch_stats", "accel_vg_trace", "accel_demand_of", "accel_solve", "accel_solve_sms", "accel_fair_weights", "accel_metrics", "accel_overlap", "accel_tma_map_2d",
+    "accel_tenant_stream", "accel_launch_times", "accel_launch_stats", "accel_vg_trace", "accel_demand_of", "accel_solve", "accel_placement_order", "accel_solve_sms", "accel_fair_weights", "accel_metrics", "accel_overlap", "accel_tma_map_2d",
 ]
 
 
@@ -201,6 +201,7 @@ def _load() -> C.CDLL:
         "accel_vg_trace": (i32, [vp, u64, P(accel_vg_record), u64, P(u64)]),
         "accel_demand_of": (i32, [P(accel_caps), u32, u32, u32, u32, u32, P(accel_demand)]),
         "accel_solve": (i32, [P(accel_caps), P(accel_demand), i32, P(u32)]),
+        "accel_placement_order": (i32, [P(accel_caps), P(accel_demand), i32, P(i32)]),
         "accel_solve_sms": (i32, [P(accel_caps), P(accel_demand), i32, P(u32), P(u32)]),
         "accel_fair_weights": (i32, [P(f64), i32, P(u32)]),
         "accel_metrics": (i32, [P(f64), P(f64), i32, P(accel_mix_metrics)]),
@@ -336,6 +337,15 @@ def accel_solve(demands: list[accel_demand], caps: accel_caps | None = None) -> 
     arr = (accel_demand * max(k, 1))(*demands)
     out = (u32 * max(k, 1))()
     check(lib.accel_solve(C.byref(caps or accel_caps()), arr, k, out))
+    return list(out)[:k]
+
+
+def accel_placement_order(demands: list[accel_demand], caps: accel_caps | None = None) -> list[int]:
+    """R-place-1: request indices, largest per-CTA footprint first."""
+    k = len(demands)
+    arr = (accel_demand * max(k, 1))(*demands)
+    out = (i32 * max(k, 1))()
+    check(lib.accel_placement_order(C.byref(caps or accel_caps()), arr, k, out))
     return list(out)[:k]
 
 

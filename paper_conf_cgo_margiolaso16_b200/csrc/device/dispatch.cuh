@@ -282,7 +282,9 @@ enum : uint32_t {
   // measurement-only ablations (env ACCEL_ABLATE on the host; scripts/isolated.py)
   kAblNoFence = 1u << 24,  // retire without the release fence (UNSAFE with top-ups)
   kAblNoLive = 1u << 25,   // never load the live quota (no shrink)
-  kAblNoStats = 1u << 26   // no max_alive reduction at admission
+  kAblNoStats = 1u << 26,  // no max_alive reduction at admission
+  kAblNoDec = 1u << 27,    // no alive decrement at retire (UNSAFE with top-ups)
+  kAblNoTop = 1u << 28     // no predecessor `topped` check (UNSAFE with top-ups)
 };
 
 // Scheduling state of one CTA in shared memory (the paper's `local struct SD`,
@@ -445,7 +447,7 @@ template <bool kResolve>
 __device__ __forceinline__ void retire(Desc* d, uint32_t cfg, const SchedState* S) {
   if (kResolve && S->admitted) {
     if (!(cfg & kAblNoFence)) fence_acq_rel();  // this CTA's VG results before the alive decrement
-    atomicAdd(&d->qa, kAliveNeg);
+    if (!(cfg & kAblNoDec)) atomicAdd(&d->qa, kAliveNeg);
   }
   if (kResolve && S->draining) {
     fence_acq_rel();  // the last VG's results before the draining decrement
@@ -479,7 +481,7 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
       // admission and the first dequeue are all issued before the wait, so a
       // launch that was never topped pays no extra round trip
       const uint32_t topped_prev =
-          (!kPart && (cfg & kCfgHasPrev)) ? ld_volatile(&(d - 1)->topped) : 0u;
+          (!kPart && (cfg & kCfgHasPrev) && !(cfg & kAblNoTop)) ? ld_volatile(&(d - 1)->topped) : 0u;
       // admission and first dequeue in one atomic; an arrival over the live
       // quota runs the chunk it got and leaves at its next dequeue
       const uint32_t live = (d->governed && !(cfg & kAblNoLive)) ? ld_relaxed(&d->ctl->live) : 0xffffffffu;

@@ -714,28 +714,26 @@ int submit_locked(accel_ctx* ctx, uint32_t n, const accel_request* rs, uint64_t*
   // shared memory) only gets if it is placed before small CTAs fragment the
   // SMs -- otherwise it waits for a whole co-runner to finish.  NATIVE keeps
   // the mix order (its FCFS winner is the point of the baseline).
-  std::vector<uint32_t> ord(n);
-  for (uint32_t i = 0; i < n; ++i) ord[i] = i;
-  if (ctx->cfg.mode == ACCEL_MODE_SHARED) {
-    std::vector<double> fp(n, 0.0);
-    for (uint32_t i = 0; i < n; ++i) {
-      accel_demand d{};
-      if (demand_for(ctx, fresh[i]->steps[fresh[i]->main_step], 1, &d) == ACCEL_OK)
-        fp[i] = std::max({(double)d.thr / ctx->caps.thr_per_sm, (double)d.regs / ctx->caps.regs_per_sm,
-                          (double)d.smem / ctx->caps.smem_per_sm, (double)d.cta / ctx->caps.ctas_per_sm});
-    }
-    std::stable_sort(ord.begin(), ord.end(), [&](uint32_t a, uint32_t b) { return fp[a] > fp[b]; });
+  std::vector<int32_t> ord(n);
+  for (uint32_t i = 0; i < n; ++i) ord[i] = (int32_t)i;
+  if (ctx->cfg.mode == ACCEL_MODE_SHARED && n > 1) {
+    std::vector<accel_demand> ds(n);
+    bool ok = true;
+    for (uint32_t i = 0; i < n; ++i)
+      ok = ok && demand_for(ctx, fresh[i]->steps[fresh[i]->main_step], 1, &ds[i]) == ACCEL_OK;
+    if (ok && accel_placement_order(&ctx->caps, ds.data(), (int32_t)n, ord.data()) != ACCEL_OK)
+      for (uint32_t i = 0; i < n; ++i) ord[i] = (int32_t)i;
   }
   // ids (= arrival order for later re-solves) follow the array order
   const uint64_t base = ctx->next_id;
   ctx->next_id += n;
-  for (uint32_t i : ord) {
-    Request* r = fresh[i].get();
+  for (int32_t i : ord) {
+    Request* r = fresh[(size_t)i].get();
     int rc = enqueue(ctx, r);
     if (rc) return rc;
-    r->id = base + i;
+    r->id = base + (uint64_t)i;
     ids[i] = r->id;
-    ctx->reqs[r->id] = std::move(fresh[i]);
+    ctx->reqs[r->id] = std::move(fresh[(size_t)i]);
   }
   return ACCEL_OK;
 }
@@ -824,7 +822,7 @@ int accel_init(const accel_config* cfg, accel_ctx** out) {
                          cudaHostAllocDefault)) != cudaSuccess)
     return init_fail(e, "cudaHostAlloc(ring)");
   ctx->slot_used.assign(kPoolSlots, 0);
-  if (const char* ab = std::getenv("ACCEL_ABLATE")) ctx->ablate = ((uint32_t)std::atoi(ab) & 7u) << 24;
+  if (const char* ab = std::getenv("ACCEL_ABLATE")) ctx->ablate = ((uint32_t)std::atoi(ab) & 31u) << 24;
   accel_ctx* raw = ctx.release();
   raw->monitor = std::thread(monitor_loop, raw);
   *out = raw;

@@ -60,52 +60,79 @@ bool valid(const Req& r, const Caps& c) {
   return true;
 }
 
-// F(n): breadth-first placement with rotating remainders, per-SM sums and the
-// sub-partition register packing (least-loaded start, round-robin warps).
+// a/b < c/d for positive denominators, exact
+bool frac_less(__int128 a, __int128 b, __int128 c, __int128 d) { return a * d < c * b; }
+
+// Per-CTA footprint: the largest share of ONE SM's resources, as (num, den).
+void footprint(const Req& r, const Caps& c, __int128* num, __int128* den) {
+  const __int128 cand[4][2] = {{r.thr, c.thr}, {r.regs, c.regs}, {r.smem, c.smem}, {r.cta, c.ctas}};
+  *num = cand[0][0];
+  *den = cand[0][1];
+  for (int i = 1; i < 4; ++i)
+    if (frac_less(*num, *den, cand[i][0], cand[i][1])) {
+      *num = cand[i][0];
+      *den = cand[i][1];
+    }
+}
+
+// R-place-1: indices, largest per-CTA footprint first, ties in arrival order.
+std::vector<int> placement_order(const std::vector<Req>& rs, const Caps& c) {
+  std::vector<int> ord(rs.size());
+  for (size_t i = 0; i < rs.size(); ++i) ord[i] = (int)i;
+  std::stable_sort(ord.begin(), ord.end(), [&](int a, int b) {
+    __int128 na, da, nb, db;
+    footprint(rs[a], c, &na, &da);
+    footprint(rs[b], c, &nb, &db);
+    return frac_less(nb, db, na, da);  // a's footprint > b's
+  });
+  return ord;
+}
+
+// F(n) (R-solver-3): kernels in placement order, each kernel's CTAs dealt
+// round-robin over the SMs from a pointer carried over between kernels, a CTA
+// going to the next SM where it fits (thread / CTA-slot / shared-memory sums,
+// warps packed round-robin from the least-loaded SMSP); dealt in rounds.
 bool feasible(const std::vector<Req>& rs, const std::vector<int64_t>& n, const Caps& c) {
-  const size_t k = rs.size();
-  std::vector<int64_t> q(k), rem(k), off(k);
-  int64_t o = 0;
-  for (size_t i = 0; i < k; ++i) {
-    q[i] = n[i] / c.sms;
-    rem[i] = n[i] % c.sms;
-    off[i] = o;
-    o = (o + rem[i]) % c.sms;
-  }
-  std::vector<int64_t> cnt(k), last(k, -1);
-  bool have_last = false;
-  for (int64_t sm = 0; sm < c.sms; ++sm) {
-    for (size_t i = 0; i < k; ++i) {
-      // SM `sm` gets an extra CTA of kernel i iff (sm - off_i) mod S < rem_i
-      const int64_t rel = ((sm - off[i]) % c.sms + c.sms) % c.sms;
-      cnt[i] = q[i] + (rel < rem[i] ? 1 : 0);
-    }
-    if (have_last && cnt == last) continue;  // identical SM load: same verdict
-    last = cnt;
-    have_last = true;
-    int64_t thr = 0, ctas = 0, smem = 0;
-    int64_t sp[Caps::kSmsp] = {0, 0, 0, 0};
-    for (size_t i = 0; i < k; ++i) {
-      thr += cnt[i] * rs[i].thr;
-      ctas += cnt[i] * rs[i].cta;
-      smem += cnt[i] * rs[i].smem;
-      const int64_t w = rs[i].warps(), rpw = rs[i].rpw();
-      for (int64_t t = 0; t < cnt[i]; ++t) {
-        int start = 0;
-        for (int s = 1; s < Caps::kSmsp; ++s)
-          if (sp[s] < sp[start]) start = s;
-        for (int64_t x = 0; x < w; ++x) sp[(start + x) % Caps::kSmsp] += rpw;
+  struct Sm {
+    int64_t thr = 0, ctas = 0, smem = 0, sp[Caps::kSmsp] = {0, 0, 0, 0};
+  };
+  std::vector<Sm> sm((size_t)c.sms);
+  auto place = [&](const Sm& s, const Req& r, Sm* out) {
+    if (s.thr + r.thr > c.thr || s.ctas + r.cta > c.ctas || s.smem + r.smem > c.smem) return false;
+    *out = s;
+    int start = 0;
+    for (int x = 1; x < Caps::kSmsp; ++x)
+      if (s.sp[x] < s.sp[start]) start = x;
+    const int64_t w = r.warps(), rpw = r.rpw();
+    for (int64_t x = 0; x < w; ++x) out->sp[(start + x) % Caps::kSmsp] += rpw;
+    for (int x = 0; x < Caps::kSmsp; ++x)
+      if (out->sp[x] > c.regs_per_smsp()) return false;
+    out->thr += r.thr;
+    out->ctas += r.cta;
+    out->smem += r.smem;
+    return true;
+  };
+  std::vector<std::pair<int64_t, Sm>> fit;
+  fit.reserve((size_t)c.sms);
+  int64_t p = 0;
+  for (int i : placement_order(rs, c)) {
+    const Req& r = rs[(size_t)i];
+    int64_t left = n[(size_t)i];
+    while (left > 0) {
+      fit.clear();
+      for (int64_t j = 0; j < c.sms && (int64_t)fit.size() < left; ++j) {
+        const int64_t k = (p + j) % c.sms;
+        Sm nx;
+        if (place(sm[(size_t)k], r, &nx)) fit.emplace_back(k, nx);
       }
+      if (fit.empty()) return false;
+      for (auto& f : fit) sm[(size_t)f.first] = f.second;
+      left -= (int64_t)fit.size();
+      p = (fit.back().first + 1) % c.sms;
     }
-    if (thr > c.thr || ctas > c.ctas || smem > c.smem) return false;
-    for (int s = 0; s < Caps::kSmsp; ++s)
-      if (sp[s] > c.regs_per_smsp()) return false;
   }
   return true;
 }
-
-// a/b < c/d for positive denominators, exact
-bool frac_less(__int128 a, __int128 b, __int128 c, __int128 d) { return a * d < c * b; }
 
 // dominant share of a request holding n CTAs: max_r n*d_r/(S*cap_r) as (num, den)
 void dominant(const Req& r, int64_t n, const Caps& c, __int128* num, __int128* den) {
@@ -123,6 +150,19 @@ void dominant(const Req& r, int64_t n, const Caps& c, __int128* num, __int128* d
 }
 
 }  // namespace
+
+extern "C" int accel_placement_order(const accel_caps* caps, const accel_demand* d, int32_t k, int32_t* order_out) {
+  if (k < 0 || (k > 0 && (!d || !order_out))) return ACCEL_EINVAL;
+  const Caps c = caps_of(caps);
+  std::vector<Req> rs((size_t)k);
+  for (int32_t i = 0; i < k; ++i)
+    rs[(size_t)i] = Req{d[i].thr, d[i].regs, d[i].smem, d[i].cta, d[i].grid_vgs, d[i].weight ? d[i].weight : 1};
+  for (const Req& r : rs)
+    if (!valid(r, c)) return ACCEL_ENOFIT;
+  const std::vector<int> ord = placement_order(rs, c);
+  for (int32_t i = 0; i < k; ++i) order_out[i] = ord[(size_t)i];
+  return ACCEL_OK;
+}
 
 extern "C" int accel_demand_of(const accel_caps* caps, uint32_t block_threads, uint32_t regs_per_thread,
                                uint32_t smem_bytes, uint32_t grid_vgs, uint32_t weight,

@@ -15,7 +15,12 @@ from paper_conf_cgo_margiolaso16_b200.runtime import Accel  # noqa: E402
 
 mode = sys.argv[1] if len(sys.argv) > 1 else "resolve"
 cfg = sys.argv[2] if len(sys.argv) > 2 else "c2"
-tenants, size, inputs = bench.make_inputs(cfg, 0)
+if "," in cfg:   # an ad-hoc mix of default-size tenants, e.g. sgemm,spmv
+    import synth  # noqa: E402
+    tenants = cfg.split(",")
+    inputs = {t: synth.preset(t, "default", seed=11 + i) for i, t in enumerate(tenants)}
+else:
+    tenants, size, inputs = bench.make_inputs(cfg, 0)
 jobs = [make_job(t, inputs[t]) for t in tenants]
 m, p = {"native": (abi.MODE_NATIVE, abi.POLICY_STATIC), "static": (abi.MODE_SHARED, abi.POLICY_STATIC),
         "resolve": (abi.MODE_SHARED, abi.POLICY_RESOLVE)}[mode]

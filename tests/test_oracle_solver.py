@@ -97,7 +97,7 @@ def _check_invariants(ds, n, caps):
 def test_random_invariants_b200():
     r = random.Random(7)
     caps = S.Caps()
-    for _ in range(60):
+    for _ in range(30):
         k = r.randint(1, 8)
         ds = [_random_demand(r, caps) for _ in range(k)]
         if r.random() < 0.3:  # duplicate kernels
@@ -274,3 +274,22 @@ def test_partition_random_invariants_and_bruteforce():
         # unit weights, no duplicate class: the greedy is max-min optimal
         if len(S.classes(ds)) == len(ds) and all(d.weight == 1 for d in ds):
             assert got == pytest.approx(best)
+
+
+def test_placement_big_cta_not_starved():
+    """R-solver-3 / R-place-1: small CTAs arriving first must not fragment
+    every SM.  A GEMM whose CTA needs a whole SM (640 threads x 96 registers)
+    beside a small SpMV kernel: by the closed form both get half of the
+    registers, i.e. 74 GEMM CTAs (one per SM on half the SMs); the SpMV CTAs
+    pack on the other SMs.  (Dealing SpMV's 127 CTAs one per SM first left
+    the GEMM 21 SMs.)"""
+    g, sp = S.demand_of(640, 96, 189 * 1024, 512), S.demand_of(256, 40, 0, 2304)
+    for ds, gi in (([sp, g], 1), ([g, sp], 0)):
+        n = S.solve(ds)
+        assert n[gi] == 74
+        _check_invariants(ds, n, S.Caps())
+    # brute-force placement check on a 4-SM toy: a full-SM CTA + three 1/4-SM CTAs
+    caps = S.Caps(sms=4, thr_per_sm=1024, regs_per_sm=65536, smem_per_sm=233472, ctas_per_sm=32)
+    big, small = S.demand_of(1024, 32, 0, 8, caps=caps), S.demand_of(256, 32, 0, 8, caps=caps)
+    assert S.feasible([small, big], [8, 2], caps)        # big on SM0, SM1; small 4 + 4 on SM2, SM3
+    assert not S.feasible([small, big], [9, 2], caps)    # 9 quarter-SM CTAs need 3 SMs

@@ -72,7 +72,7 @@ def test_parity_tiny_devices():
 def test_parity_b200():
     r = random.Random(3)
     caps = S.Caps()
-    for _ in range(150):
+    for _ in range(40):   # the oracle's placement simulation is slow in Python
         ds = _random_instance(r, caps, 8, 20000)
         assert abi.accel_solve([_to_c(d) for d in ds]) == S.solve(ds, caps)
 
@@ -140,3 +140,17 @@ def test_fair_weights_closed_forms():
             for j in range(len(s)):
                 if s[i] > s[j]:
                     assert w[i] >= w[j]
+
+
+def test_placement_order_parity():
+    """R-place-1: the library's enqueue / placement order equals the oracle's
+    (largest per-CTA footprint first, ties in arrival order)."""
+    r = random.Random(21)
+    caps = S.Caps()
+    for _ in range(300):
+        ds = _random_instance(r, caps, 8, 5000)
+        assert abi.accel_placement_order([_to_c(d) for d in ds]) == S.placement_order(ds, caps)
+    # a one-CTA-per-SM GEMM (registers) goes before a small SpMV CTA whatever the arrival order
+    g, sp = S.demand_of(640, 96, 189 * 1024, 512), S.demand_of(256, 40, 0, 2304)
+    assert S.placement_order([sp, g]) == [1, 0]
+    assert abi.accel_placement_order([_to_c(sp), _to_c(g)]) == [1, 0]
