@@ -72,7 +72,10 @@ def test_staggered_multi_launch_mix(racc, oracle_lib, seed):
     or grows the others, multi-launch requests (bfs levels, histo iterations,
     stencil sweeps) stay correct."""
     from paper_conf_cgo_margiolaso16_b200.jobs import BfsJob, HistoJob, StencilJob, TpacfJob
-    dsn = synth.preset("stencil", "default", seed=seed, sweeps=30)
+    # the stencil (100 sweeps, ~3.5 ms) is still running when every later
+    # request arrives (~1 ms of host time per submission), so each arrival
+    # must re-solve it
+    dsn = synth.preset("stencil", "default", seed=seed, sweeps=100)
     dbf = synth.preset("bfs", "default", seed=seed)
     dhi = synth.preset("histo", "default", seed=seed, iters=8)
     dtp = synth.preset("tpacf", "small", seed=seed)
@@ -85,13 +88,11 @@ def test_staggered_multi_launch_mix(racc, oracle_lib, seed):
     st = [racc.stats(i) for i in ids]
     racc.release()
     assert all(s.coverage_ok == 1 for s in st)
-    assert sum(s.resolves for s in st) >= 1
+    assert st[0].resolves >= 1
     assert np.array_equal(jobs[1].result()["level"], oracle_lib.bfs(dbf)[0])
     assert np.array_equal(jobs[2].result()["counts"], oracle_lib.histo(dhi)[0])
     dd, rr, dr = oracle_lib.tpacf(dtp)
     r = jobs[3].result()
     assert np.array_equal(r["dd"], dd) and np.array_equal(r["rr"], rr) and np.array_equal(r["dr"], dr)
-    zlo, zhi = 10, 54  # planes 40..43 depend on [10, 74) ∩ [0, 64) after 30 sweeps
-    slab = dict(dsn, a0=np.ascontiguousarray(dsn["a0"][zlo:]), nz=64 - zlo)
-    ref = oracle_lib.stencil(slab)
-    assert_close_fp32(jobs[0].result()["a"][40:44], ref[40 - zlo:44 - zlo], what="stencil")
+    ref = oracle_lib.stencil(dsn)   # full volume (100 sweeps reach every plane)
+    assert_close_fp32(jobs[0].result()["a"][38:46], ref[38:46], what="stencil")
