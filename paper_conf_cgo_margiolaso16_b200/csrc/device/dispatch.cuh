@@ -279,6 +279,9 @@ enum : uint32_t {
   kCfgStamps = 1u << 17,
   kCfgHasPrev = 1u << 18,  // the request ran a launch before this one (RESOLVE
                            // persistent grids check its `topped` word)
+  kCfgStaticFirst = 1u << 19,  // main grid: CTA b's first chunk is [b*chunk, (b+1)*chunk)
+                               // with no atomic (desc_init starts the queue head at
+                           // grid*chunk and, under RESOLVE, `alive` at grid)
   // measurement-only ablations (env ACCEL_ABLATE on the host; scripts/isolated.py)
   kAblNoFence = 1u << 24,  // retire without the release fence (UNSAFE with top-ups)
   kAblNoLive = 1u << 25,   // never load the live quota (no shrink)
@@ -468,8 +471,12 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     S->admitted = 1;
     S->draining = 0;
     S->over = 0;
+    // Static first chunk (main grids): measured, the first dequeue of 740
+    // CTAs on one queue word serialised in L2 and spread the CTAs' first VG
+    // starts over 6 us of a 30-us stencil launch (scripts/vg_trace.py)
+    const bool stat = (cfg & kCfgStaticFirst) != 0u;
     if (!kResolve) {
-      b = qa_next(atomicAdd(&d->qa, (unsigned long long)chunk));   // issued before anything else
+      b = stat ? blockIdx.x * chunk : qa_next(atomicAdd(&d->qa, (unsigned long long)chunk));
     } else if (kPart && part_leave(S->owner, d->ctl, S->sm, S->tok, S->hint_owner, S->hint_q, S->hint_c)) {
       // PARTITION: the SM was handed over between two launches: leave unadmitted
       S->left = 1;
@@ -485,18 +492,28 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
       // admission and first dequeue in one atomic; an arrival over the live
       // quota runs the chunk it got and leaves at its next dequeue
       const uint32_t live = (d->governed && !(cfg & kAblNoLive)) ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
-      const unsigned long long v = atomicAdd(&d->qa, kAlive1 | chunk);
-      b = qa_next(v);
-      const uint32_t a = qa_alive(v) + 1u;
+      uint32_t a;
+      if (stat) {
+        // admitted from the start (alive = grid); a shrink that came first
+        // evicts at the next dequeue
+        b = blockIdx.x * chunk;
+        a = gridDim.x;
+        if (blockIdx.x == 0 && !(cfg & kAblNoStats))
+          asm volatile("red.relaxed.gpu.global.max.u32 [%0], %1;" ::"l"(&d->max_alive), "r"(a) : "memory");
+      } else {
+        const unsigned long long v = atomicAdd(&d->qa, kAlive1 | chunk);
+        b = qa_next(v);
+        a = qa_alive(v) + 1u;
+        if (!(cfg & kAblNoStats))
+          asm volatile("red.relaxed.gpu.global.max.u32 [%0], %1;" ::"l"(&d->max_alive), "r"(a) : "memory");
+        if (a > live) {
+          S->over = 1;
+          red_add_u32(&d->admit_fail, 1u);
+          d->last_live = live;
+        }
+      }
       // the CTA holding the launch's first ticket announces it to top-up grids
       if (b == 0) asm volatile("red.relaxed.gpu.global.max.u32 [%0], %1;" ::"l"(&d->ctl->cur), "r"(d->req_idx) : "memory");
-      if (!(cfg & kAblNoStats))
-        asm volatile("red.relaxed.gpu.global.max.u32 [%0], %1;" ::"l"(&d->max_alive), "r"(a) : "memory");
-      if (a > live) {
-        S->over = 1;
-        red_add_u32(&d->admit_fail, 1u);
-        d->last_live = live;
-      }
       S->hint_live = live;
       S->hint_alive = a;
       if (topped_prev) wait_complete(d - 1);

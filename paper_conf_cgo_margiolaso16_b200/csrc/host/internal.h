@@ -20,6 +20,9 @@ struct InitStep {
   uint32_t cov_offset; // coverage offset of the step's first launch
   uint32_t ctas_per_sm; // PARTITION: c_i of the step's kernel (0 otherwise)
   const uint32_t* order; // dequeue order (nullptr: linear)
+  uint64_t qa0;          // initial queue word (alive << 32 | next): main grids with
+                         // static first chunks start at grid*chunk (alive = grid
+                         // under RESOLVE); 0 otherwise
 };
 
 struct InitParams {

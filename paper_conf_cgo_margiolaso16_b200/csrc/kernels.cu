@@ -66,7 +66,7 @@ __global__ void desc_init_kernel(const InitParams p, uint32_t n_desc) {
   d->topped = p.owner != nullptr ? 1u : 0u;   // PARTITION: any grid may serve any launch
   d->req_idx = i;
   d->has_prev = i > 0 ? 1u : 0u;
-  d->qa = 0;
+  d->qa = st.qa0;
 }
 
 // Request completion: wait until the last launch completed if another grid
