@@ -491,7 +491,10 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
           (!kPart && (cfg & kCfgHasPrev) && !(cfg & kAblNoTop)) ? ld_volatile(&(d - 1)->topped) : 0u;
       // admission and first dequeue in one atomic; an arrival over the live
       // quota runs the chunk it got and leaves at its next dequeue
-      const uint32_t live = (d->governed && !(cfg & kAblNoLive)) ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
+      // (a static-first CTA reads the live quota after its first dynamic
+      // dequeue: a shrink that precedes the launch evicts one chunk later,
+      // and the launch start carries no load of the control line)
+      const uint32_t live = (d->governed && !stat && !(cfg & kAblNoLive)) ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
       uint32_t a;
       if (stat) {
         // admitted from the start (alive = grid); a shrink that came first
