@@ -207,12 +207,15 @@ def run_reference(args):
     tenants, size, inputs = make_inputs(args.config, 0)
     from oracle import tenants as O
     O.build()
+    # samples sized so that the timed steps take ~2 minutes in all (larger
+    # samples extrapolate better: tiny ones are dominated by thread start-up)
+    budget = min(3.0, max(0.3, 120.0 / max(1, args.steps) / len(tenants)))
     for _ in range(args.warmup):
         cpu_mix_seconds(tenants, inputs, 0.3)
     secs = []
     desc = ""
     for _ in range(args.steps):
-        s, desc = cpu_mix_seconds(tenants, inputs, 0.3)
+        s, desc = cpu_mix_seconds(tenants, inputs, budget)
         secs.append(s)
     ms = 1e3 * statistics.mean(secs)
     value = 1e3 / ms

@@ -165,6 +165,8 @@ def sampled(r: Runner, ta, reps, k, n, seed):
             runs = [mix_metrics(r.run(jobs, mode, pol), [ta[t] for t in names]) for _ in range(reps)]
             res[name] = {kk: statistics.mean(x[kk] for x in runs) for kk in ("U", "STP", "ANTT", "makespan_ms", "WANTT")}
         mixes.append(res)
+        print(json.dumps({"mix": names, **{nm: {kk: round(v, 3) for kk, v in res[nm].items()} for nm, _, _ in MODES}}),
+              flush=True)
     out = {}
     for name in SHARED:
         fi = [m["native"]["U"] / m[name]["U"] for m in mixes]
@@ -174,7 +176,12 @@ def sampled(r: Runner, ta, reps, k, n, seed):
                      "STP_ratio_gmean": gm([m[name]["STP"] / m["native"]["STP"] for m in mixes]),
                      "throughput_speedup_gmean": gm([m["native"]["makespan_ms"] / m[name]["makespan_ms"]
                                                      for m in mixes]),
-                     "WANTT_max": max(m[name]["WANTT"] for m in mixes)}
+                     "WANTT_max": max(m[name]["WANTT"] for m in mixes),
+                     # BASELINE.json target for 4-tenant mixes: U <= 1.5 and STP >= native
+                     "target_met_pct": 100.0 * sum(m[name]["U"] <= 1.5 and m[name]["STP"] >= m["native"]["STP"]
+                                                   for m in mixes) / len(mixes),
+                     "U_le_1.5_pct": 100.0 * sum(m[name]["U"] <= 1.5 for m in mixes) / len(mixes),
+                     "STP_ge_native_pct": 100.0 * sum(m[name]["STP"] >= m["native"]["STP"] for m in mixes) / len(mixes)}
     out["native"] = {"U_gmean": gm([m["native"]["U"] for m in mixes]),
                      "WANTT_max": max(m["native"]["WANTT"] for m in mixes)}
     return mixes, out
