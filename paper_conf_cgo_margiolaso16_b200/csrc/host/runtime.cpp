@@ -170,6 +170,19 @@ struct accel_ctx {
   // (16 main + 12 top-up + 1 control <= CUDA_DEVICE_MAX_CONNECTIONS = 32).
   static constexpr int kTopupStreams = 12;
   cudaStream_t topup[kTopupStreams] = {};
+  // a growth grid is sticky (it follows its step's later launches), so a grid
+  // queued behind another request's on the same stream would not start until
+  // that one's step ends: take an idle top-up stream when there is one
+  cudaStream_t pick_topup_stream() {
+    for (int i = 0; i < kTopupStreams; ++i) {
+      const uint32_t k = (topup_rr + (uint32_t)i) % kTopupStreams;
+      if (cudaStreamQuery(topup[k]) == cudaSuccess) {
+        topup_rr = k + 1;
+        return topup[k];
+      }
+    }
+    return topup[topup_rr++ % kTopupStreams];
+  }
   uint32_t topup_rr = 0;
   cudaStream_t ctl = nullptr;
   cudaEvent_t epoch = nullptr;
@@ -521,7 +534,7 @@ int apply_quota(accel_ctx* ctx, Request* r, uint32_t q) {
     accel::Desc* d = ctx->desc_ptr(r->slot + st.first);
     uint32_t sticky = st.repeat;
     void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &sticky};
-    cudaStream_t ts = ctx->topup[ctx->topup_rr++ % accel_ctx::kTopupStreams];
+    cudaStream_t ts = ctx->pick_topup_stream();
     CK(ctx, cudaLaunchKernel(k.tfn, dim3(q - r->provisioned, 1, 1), k.block, params, k.dyn_smem, ts));
     cudaEvent_t ev;
     CK(ctx, ctx->get_event(&ev));
@@ -558,7 +571,7 @@ int apply_sms(accel_ctx* ctx, Request* r, uint32_t sms) {
     accel::Desc* d = ctx->desc_ptr(r->slot + st.first);
     uint32_t sticky = st.repeat;
     void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &sticky};
-    cudaStream_t ts = ctx->topup[ctx->topup_rr++ % accel_ctx::kTopupStreams];
+    cudaStream_t ts = ctx->pick_topup_stream();
     CK(ctx, cudaLaunchKernel(k.partfn, dim3((sms - r->sms_provisioned) * (uint32_t)k.occ_part, 1, 1), k.block,
                              params, k.part_smem, ts));
     cudaEvent_t ev;
