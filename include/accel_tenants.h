@@ -120,14 +120,21 @@ typedef struct {
   uint32_t m, n, k;
 } accel_sgemm_args;
 
-/* sgemm_split -- tf32 split of an fp32 array for the 3xTF32 tensor-core GEMM:
- * hi = round-to-nearest tf32 of src, lo = src - hi (exact).  block 256,
- * VG = 4096 elements, grid ceil(n/4096).  16-B aligned arrays. */
+/* sgemm_split -- tf32 split of the two fp32 operands of the 3xTF32
+ * tensor-core GEMM in ONE launch: hi = round-to-nearest tf32 of src, lo =
+ * src - hi (exact), for segment 0 (A: src0/hi0/lo0, n0 elements) and
+ * segment 1 (B).  block 256, VG = 4096 elements of one segment: VGs
+ * [0, ceil(n0/4096)) split A, the next ceil(n1/4096) split B; grid = their
+ * sum.  16-B aligned arrays; n1 = 0 for a single array. */
 typedef struct {
-  const float *src;
-  float *hi;
-  float *lo;
-  uint64_t n;
+  const float *src0;
+  float *hi0;
+  float *lo0;
+  uint64_t n0;
+  const float *src1;
+  float *hi1;
+  float *lo1;
+  uint64_t n1;
 } accel_sgemm_split_args;
 
 /* sgemm_tc -- C[m][n] = A.B^T on tcgen05 tensor cores, 3xTF32

@@ -143,7 +143,8 @@ class accel_sgemm_args(C.Structure):
 
 
 class accel_sgemm_split_args(C.Structure):
-    _fields_ = [("src", vp), ("hi", vp), ("lo", vp), ("n", u64)]
+    _fields_ = [("src0", vp), ("hi0", vp), ("lo0", vp), ("n0", u64),
+                ("src1", vp), ("hi1", vp), ("lo1", vp), ("n1", u64)]
 
 
 class accel_sgemm_tc_args(C.Structure):

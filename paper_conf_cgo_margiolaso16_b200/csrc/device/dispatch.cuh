@@ -279,6 +279,9 @@ enum : uint32_t {
   kCfgStamps = 1u << 17,
   kCfgHasPrev = 1u << 18,  // the request ran a launch before this one (RESOLVE
                            // persistent grids check its `topped` word)
+  kCfgWaitPrev = 1u << 20,     // wait for the predecessor launch on the device whether or not
+                               // it was topped up (R-place-3: this grid was launched ahead
+                               // on a side stream, not behind its predecessor)
   kCfgStaticFirst = 1u << 19,  // main grid: CTA b's first chunk is [b*chunk, (b+1)*chunk)
                                // with no atomic (desc_init starts the queue head at
                            // grid*chunk and, under RESOLVE, `alive` at grid)
@@ -497,7 +500,8 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
       // admission and the first dequeue are all issued before the wait, so a
       // launch that was never topped pays no extra round trip
       const uint32_t topped_prev =
-          (!kPart && (cfg & kCfgHasPrev) && !(cfg & kAblNoTop)) ? ld_volatile(&(d - 1)->topped) : 0u;
+          (cfg & kCfgWaitPrev) ? 1u
+          : (!kPart && (cfg & kCfgHasPrev) && !(cfg & kAblNoTop)) ? ld_volatile(&(d - 1)->topped) : 0u;
       // admission and first dequeue in one atomic; an arrival over the live
       // quota runs the chunk it got and leaves at its next dequeue
       // (a static-first CTA reads the live quota after its first dynamic

@@ -98,6 +98,9 @@ struct Request {
   uint32_t quota_initial = 0, quota_min = 0, quota_max = 0, resolves = 0;
   size_t enq_step = 0;       // enqueue cursor (enqueue_next)
   uint32_t enq_launch = 0, enq_li = 0;
+  bool early_main = false;   // R-place-3: main step launched ahead on a side stream
+  uint32_t early_sms = 0;    // SMs its waiting grid may hold (released when done)
+  cudaEvent_t ev_early = nullptr;  // recorded after that launch (the main stream waits for it)
   uint32_t live = 0;         // RESOLVE: current live quota of the main step
   uint32_t provisioned = 0;  // RESOLVE: main-grid CTAs + sticky top-up CTAs
   bool part = false;         // PARTITION request
@@ -168,6 +171,7 @@ struct accel_ctx {
   // RESOLVE top-up grids are sticky (they follow a request's launches), so two
   // of them must never share a stream: a pool with its own hardware queues
   // (16 main + 12 top-up + 1 control <= CUDA_DEVICE_MAX_CONNECTIONS = 32).
+  uint32_t early_sms = 0;   // R-place-3: SMs held by early grids still waiting on the device
   static constexpr int kTopupStreams = 12;
   cudaStream_t topup[kTopupStreams] = {};
   // a growth grid is sticky (it follows its step's later launches), so a grid
@@ -254,6 +258,8 @@ int refresh_done(accel_ctx* ctx, Request* r) {
   for (size_t i = 0; e == cudaSuccess && i < r->ev_topups.size(); ++i) e = cudaEventQuery(r->ev_topups[i]);
   if (e == cudaSuccess) {
     r->done = true;
+    ctx->early_sms -= r->early_sms;
+    r->early_sms = 0;
   } else if (e != cudaErrorNotReady) {
     return ctx->cuda(e, "cudaEventQuery");
   }
@@ -357,6 +363,47 @@ int enqueue_begin(accel_ctx* ctx, Request* r) {
   r->enq_step = 0;
   r->enq_launch = 0;
   r->enq_li = 0;
+  // R-place-3: a request whose main step is its last, single launch of CTAs
+  // that take at least half an SM (the tensor-core GEMM after its operand
+  // split) launches that grid NOW, on a side stream, so the block scheduler
+  // places it before the co-runners' small CTAs fragment every SM; its CTAs
+  // wait on the device for the earlier steps (kCfgWaitPrev).  RESOLVE only
+  // (the wait needs the alive accounting) and only with a quota below the
+  // SM count (a quota holding every SM would leave the earlier steps nowhere
+  // to run).
+  r->early_main = false;
+  const size_t ms = (size_t)r->main_step;
+  if (shared && !part && resolve && ms > 0 && ms + 1 == r->steps.size() && r->steps[ms].repeat == 1 &&
+      // the early grids' CTAs wait on the device while holding (up to) an SM
+      // each: together they may hold at most half the device, so the earlier
+      // steps and every co-runner always have SMs to make progress on (two
+      // early GEMMs of 74 CTAs each would otherwise hold all 148 SMs and wait
+      // for split steps that can run nowhere)
+      ctx->early_sms + r->steps[ms].quota <= (uint32_t)ctx->caps.sms / 2) {
+    const Step& st = r->steps[ms];
+    const Kernel& k = ctx->kernels[st.kid];
+    accel_demand dm{};
+    if (demand_for(ctx, st, 1, &dm) == ACCEL_OK &&
+        (2 * (int64_t)dm.thr >= ctx->caps.thr_per_sm || 2 * (int64_t)dm.regs >= ctx->caps.regs_per_sm ||
+         2 * (int64_t)dm.smem >= ctx->caps.smem_per_sm)) {
+      r->early_main = true;
+      r->early_sms = st.quota;
+      ctx->early_sms += st.quota;
+      cudaEvent_t ev_init;
+      CK(ctx, ctx->get_event(&ev_init));
+      CK(ctx, cudaEventRecord(ev_init, s));            // descriptors initialised
+      cudaStream_t es = ctx->pick_topup_stream();
+      CK(ctx, cudaStreamWaitEvent(es, ev_init, 0));
+      ctx->free_events.push_back(ev_init);             // reusable once recorded + waited on
+      accel::Desc* d = ctx->desc_ptr(r->slot + st.first);
+      // kCfgResolve | kCfgStamps | kCfgHasPrev | kCfgStaticFirst | kCfgWaitPrev
+      uint32_t cfg = (k.chunk & 0xffffu) | (1u << 16) | (1u << 17) | (1u << 18) | (1u << 19) | (1u << 20) | ctx->ablate;
+      void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &cfg};
+      CK(ctx, cudaLaunchKernel(k.prfn, dim3(st.quota, 1, 1), k.block, params, k.dyn_smem, es));
+      CK(ctx, ctx->get_event(&r->ev_early));
+      CK(ctx, cudaEventRecord(r->ev_early, es));
+    }
+  }
   return ACCEL_OK;
 }
 
@@ -367,7 +414,8 @@ int enqueue_next(accel_ctx* ctx, Request* r, bool* more) {
   const bool resolve = shared && (is_resolve(ctx->cfg.policy) || part);
   const bool lev = (r->flags & ACCEL_REQ_LAUNCH_EVENTS) != 0;
   cudaStream_t s = ctx->main[r->tenant];
-  if (r->enq_step >= r->steps.size()) {
+  const size_t n_units = r->early_main ? (size_t)r->main_step : r->steps.size();
+  if (r->enq_step >= n_units) {
     *more = false;
     return ACCEL_OK;
   }
@@ -402,7 +450,7 @@ int enqueue_next(accel_ctx* ctx, Request* r, bool* more) {
       r->enq_step += 1;
     }
   }
-  *more = r->enq_step < r->steps.size();
+  *more = r->enq_step < n_units;
   return ACCEL_OK;
 }
 
@@ -411,6 +459,13 @@ int enqueue_end(accel_ctx* ctx, Request* r) {
   const bool part = shared && r->part;
   const bool resolve = shared && (is_resolve(ctx->cfg.policy) || part);
   cudaStream_t s = ctx->main[r->tenant];
+  if (r->early_main) {
+    // launch-time stamps: the early grid's work starts once the earlier
+    // steps are complete, i.e. here on the main stream
+    if (r->flags & ACCEL_REQ_LAUNCH_EVENTS) CK(ctx, cudaEventRecord(r->ev_launch[r->enq_li], s));
+    CK(ctx, cudaStreamWaitEvent(s, r->ev_early, 0));
+    r->enq_li = r->n_desc;   // the early launch was the last one
+  }
   if (r->flags & ACCEL_REQ_LAUNCH_EVENTS) CK(ctx, cudaEventRecord(r->ev_launch[r->enq_li], s));
   if (resolve) CK(ctx, accel::launch_join(ctx->desc_ptr(r->slot + r->n_desc - 1), part ? kOwnerWords : 0u, s));
   for (const accel_copy& c : r->d2h) CK(ctx, cudaMemcpyAsync(c.dst, c.src, c.bytes, cudaMemcpyDeviceToHost, s));
@@ -528,7 +583,9 @@ int apply_quota(accel_ctx* ctx, Request* r, uint32_t q) {
   uint32_t* h = ctx->pinned_ring + (ctx->ring_pos++ % kRing);
   *h = q;
   CK(ctx, cudaMemcpyAsync(ctx->ctl_pool + (size_t)r->slot * kCtlBytes /* Ctl::live */, h, sizeof(uint32_t), cudaMemcpyHostToDevice, ctx->ctl));
-  if (q > r->provisioned) {
+  // (no growth grids for an early main step: they would wait beside it for
+  // the earlier steps and could hold the SMs those need)
+  if (q > r->provisioned && !r->early_main) {
     const Step& st = r->steps[r->main_step];
     const Kernel& k = ctx->kernels[st.kid];
     accel::Desc* d = ctx->desc_ptr(r->slot + st.first);
@@ -831,6 +888,7 @@ void release_request(accel_ctx* ctx, Request* r) {
   if (r->trace) cudaFree(r->trace);
   if (r->ev_arrival) ctx->free_events.push_back(r->ev_arrival);
   if (r->ev_done) ctx->free_events.push_back(r->ev_done);
+  if (r->ev_early) ctx->free_events.push_back(r->ev_early);
   for (cudaEvent_t ev : r->ev_launch) ctx->free_events.push_back(ev);
   for (cudaEvent_t ev : r->ev_topups) ctx->free_events.push_back(ev);
 }

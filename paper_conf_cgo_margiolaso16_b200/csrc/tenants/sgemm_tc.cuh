@@ -5,7 +5,7 @@
 //   C = A_hi.B_hi + A_hi.B_lo + A_lo.B_hi      (fp32 accumulation in TMEM)
 // 1xTF32 alone (10-bit mantissa) would miss the 1e-4 bound (~1e-3 error).
 //
-// Request = three steps: sgemm_split(A), sgemm_split(B), sgemm_tc.
+// Request = two steps: sgemm_split (A and B in one launch), sgemm_tc.
 // sgemm_tc VG = one 128 x 256 tile of C; 640 threads (20 warps):
 //   warp 0 lane 0  TMA producer  (4 tiles per 32-wide K slab, 2-stage ring, mbarriers)
 //   warp 1 lane 0  MMA issuer    (12 x tcgen05.mma 128x256x8 per slab, commit frees the slot)
@@ -73,20 +73,27 @@ struct SgemmSplit {
     return __uint_as_float(h);
   }
   static __device__ __forceinline__ void body(const Args& a, const VirtualBlock& vb, char*) {
-    const uint64_t base = (uint64_t)vb.linear * kPerVG;
+    // VGs [0, g0) split segment 0 (A), the rest segment 1 (B)
+    const uint32_t g0 = (uint32_t)((a.n0 + kPerVG - 1) / kPerVG);
+    const bool s1 = vb.linear >= g0;
+    const float* __restrict__ src = s1 ? a.src1 : a.src0;
+    float* __restrict__ hi = s1 ? a.hi1 : a.hi0;
+    float* __restrict__ lo = s1 ? a.lo1 : a.lo0;
+    const uint64_t n = s1 ? a.n1 : a.n0;
+    const uint64_t base = (uint64_t)(s1 ? vb.linear - g0 : vb.linear) * kPerVG;
 #pragma unroll
     for (int u = 0; u < 4; ++u) {
       const uint64_t i = base + (uint64_t)(u * kThreads + threadIdx.x) * 4;
-      if (i + 3 < a.n) {
-        const float4 v = __ldcs(reinterpret_cast<const float4*>(a.src + i));
+      if (i + 3 < n) {
+        const float4 v = __ldcs(reinterpret_cast<const float4*>(src + i));
         const float4 h = make_float4(hi_of(v.x), hi_of(v.y), hi_of(v.z), hi_of(v.w));
-        *reinterpret_cast<float4*>(a.hi + i) = h;
-        *reinterpret_cast<float4*>(a.lo + i) = make_float4(v.x - h.x, v.y - h.y, v.z - h.z, v.w - h.w);
+        *reinterpret_cast<float4*>(hi + i) = h;
+        *reinterpret_cast<float4*>(lo + i) = make_float4(v.x - h.x, v.y - h.y, v.z - h.z, v.w - h.w);
       } else {
-        for (uint64_t j = i; j < a.n && j < i + 4; ++j) {
-          const float h = hi_of(a.src[j]);
-          a.hi[j] = h;
-          a.lo[j] = a.src[j] - h;
+        for (uint64_t j = i; j < n && j < i + 4; ++j) {
+          const float h = hi_of(src[j]);
+          hi[j] = h;
+          lo[j] = src[j] - h;
         }
       }
     }

@@ -396,7 +396,7 @@ class SgemmJob(Job):
 
 
 class SgemmTcJob(Job):
-    """sgemm on the tcgen05 tensor cores (3xTF32): steps split(A), split(B), tc."""
+    """sgemm on the tcgen05 tensor cores (3xTF32): steps split(A and B), tc."""
 
     def __init__(self, d: dict, device="cuda"):
         super().__init__(name="sgemm", device=torch.device(device))
@@ -416,14 +416,14 @@ class SgemmTcJob(Job):
         self.c = torch.empty(m * n, dtype=torch.float32, device=self.device)
         self.out = {"c": self.c}
         s = self.split
-        self.args_sa = abi.accel_sgemm_split_args(self.inputs["a"].data_ptr(), s["a_hi"].data_ptr(),
-                                                  s["a_lo"].data_ptr(), m * k)
-        self.args_sb = abi.accel_sgemm_split_args(self.inputs["b"].data_ptr(), s["b_hi"].data_ptr(),
-                                                  s["b_lo"].data_ptr(), n * k)
+        # one launch splits both operands (VGs of A first, then of B)
+        self.args_s = abi.accel_sgemm_split_args(self.inputs["a"].data_ptr(), s["a_hi"].data_ptr(),
+                                                 s["a_lo"].data_ptr(), m * k,
+                                                 self.inputs["b"].data_ptr(), s["b_hi"].data_ptr(),
+                                                 s["b_lo"].data_ptr(), n * k)
         self.args_tc = abi.accel_sgemm_tc_args(self.tmaps.data_ptr(), self.c.data_ptr(), m, n, k)
-        self.main_step = 2
-        self.steps = [Step("sgemm_split", (_cdiv(m * k, 4096), 1, 1), self.args_sa, 1),
-                      Step("sgemm_split", (_cdiv(n * k, 4096), 1, 1), self.args_sb, 1),
+        self.main_step = 1
+        self.steps = [Step("sgemm_split", (_cdiv(m * k, 4096) + _cdiv(n * k, 4096), 1, 1), self.args_s, 1),
                       Step("sgemm_tc", (_cdiv(n, 256), _cdiv(m, 128), 1), self.args_tc, 1)]
 
     def result(self):

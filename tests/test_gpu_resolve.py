@@ -96,3 +96,27 @@ def test_staggered_multi_launch_mix(racc, oracle_lib, seed):
     assert np.array_equal(r["dd"], dd) and np.array_equal(r["rr"], rr) and np.array_equal(r["dr"], dr)
     ref = oracle_lib.stencil(dsn)   # full volume (100 sweeps reach every plane)
     assert_close_fp32(jobs[0].result()["a"][38:46], ref[38:46], what="stencil")
+
+
+@pytest.mark.parametrize("partner", ["spmv", "sgemm", "cutcp"])
+def test_early_gemm_placement(racc, oracle_lib, partner):
+    """R-place-3: the tensor-core GEMM (one CTA per SM) is launched ahead of
+    its split steps and waits for them on the device.  Results stay exact,
+    every VG runs once, and two such requests together (their early grids
+    would hold every SM) still complete: the second one is not launched early."""
+    from paper_conf_cgo_margiolaso16_b200.jobs import make_job
+    d = synth.preset("sgemm", "default", seed=3)
+    dp = synth.preset(partner, "default", seed=4)
+    jobs = [make_job("sgemm", d), make_job(partner, dp)]
+    st = racc.run(jobs)
+    assert all(s.coverage_ok == 1 for s in st)
+    r = np.random.Generator(np.random.PCG64(5))
+    ij = np.stack([r.integers(0, d["m"], 2000), r.integers(0, d["n"], 2000)], 1)
+    assert_close_fp32(jobs[0].result()["c"][ij[:, 0], ij[:, 1]], oracle_lib.sgemm_entries(d, ij), what="sgemm")
+    if partner == "sgemm":
+        assert_close_fp32(jobs[1].result()["c"][ij[:, 0], ij[:, 1]], oracle_lib.sgemm_entries(dp, ij),
+                          what="sgemm partner")
+    elif partner == "spmv":
+        assert_close_fp32(jobs[1].result()["y"], oracle_lib.spmv(dp), what="spmv")
+    # the GEMM kept its solved share: 74 CTAs (half the SMs) beside one partner
+    assert st[0].quota_initial >= 37
