@@ -207,6 +207,12 @@ typedef struct {
   uint64_t vgs_hint;          /* FAIR: VGs the request will run; 0 = the sum of
                                  its static grids (dynamic-total kernels such as
                                  bfs run fewer: pass 0 AND isolated_ns = 0)     */
+  const float *progress_weights; /* FAIR, optional (HOST, copied at submit):
+                                 relative cost of the request's VGs in the order
+                                 they are dequeued (launch by launch, ticket
+                                 order), so that progress = cost share of the
+                                 VGs done rather than their count; NULL = equal */
+  uint64_t n_progress_weights; /* entries in progress_weights (== vgs_hint)     */
 } accel_request;
 
 /* Submit one request (solver run over the active set incl. this one).

@@ -77,7 +77,8 @@ class accel_request(C.Structure):
     _fields_ = [("tenant", i32), ("flags", u32), ("weight", u32), ("main_step", i32), ("n_steps", u32), ("steps", C.POINTER(accel_launch)),
                 ("n_clear", u32), ("clear", C.POINTER(accel_clear)), ("n_h2d", u32),
                 ("h2d", C.POINTER(accel_copy)), ("n_d2h", u32), ("d2h", C.POINTER(accel_copy)),
-                ("isolated_ns", u64), ("vgs_hint", u64)]
+                ("isolated_ns", u64), ("vgs_hint", u64),
+                ("progress_weights", vp), ("n_progress_weights", u64)]
 
 
 class accel_req_stats(C.Structure):

@@ -106,6 +106,8 @@ struct Request {
   bool part = false;         // PARTITION request
   uint64_t iso_ns = 0;       // FAIR: isolated-time hint (0: none)
   uint64_t vgs_hint = 0;     // FAIR: VGs the request runs
+  std::vector<double> cum_w; // FAIR: prefix sums of the progress weights (empty: count VGs)
+  cudaEvent_t ev_start = nullptr;  // FAIR: before the first launch (device-time elapsed)
   std::chrono::steady_clock::time_point t_submit;
   uint32_t done_vgs = 0;     // FAIR: last progress read
   uint32_t sms = 0;          // PARTITION: current SM quota
@@ -172,6 +174,7 @@ struct accel_ctx {
   // of them must never share a stream: a pool with its own hardware queues
   // (16 main + 12 top-up + 1 control <= CUDA_DEVICE_MAX_CONNECTIONS = 32).
   uint32_t early_sms = 0;   // R-place-3: SMs held by early grids still waiting on the device
+  cudaEvent_t ev_now = nullptr;  // FAIR: "now" on the control stream
   static constexpr int kTopupStreams = 12;
   cudaStream_t topup[kTopupStreams] = {};
   // a growth grid is sticky (it follows its step's later launches), so a grid
@@ -356,6 +359,10 @@ int enqueue_begin(accel_ctx* ctx, Request* r) {
                                  shared ? st.order : nullptr, qa0};
   }
   CK(ctx, accel::launch_desc_init(p, r->n_desc, s));
+  if (shared && ctx->cfg.policy == ACCEL_POLICY_FAIR && r->iso_ns) {
+    CK(ctx, ctx->get_event(&r->ev_start));
+    CK(ctx, cudaEventRecord(r->ev_start, s));
+  }
   if (r->flags & ACCEL_REQ_LAUNCH_EVENTS) {
     r->ev_launch.resize(r->n_desc + 1);
     for (auto& ev : r->ev_launch) CK(ctx, ctx->get_event(&ev));
@@ -556,6 +563,12 @@ int build_request(accel_ctx* ctx, const accel_request& in, std::unique_ptr<Reque
     for (const Step& s : r->steps) vgs += (uint64_t)s.total * s.repeat;
     r->vgs_hint = in.vgs_hint ? in.vgs_hint : vgs;
   }
+  if (in.progress_weights && in.n_progress_weights) {
+    r->cum_w.assign(in.n_progress_weights + 1, 0.0);
+    for (uint64_t i = 0; i < in.n_progress_weights; ++i)
+      r->cum_w[i + 1] = r->cum_w[i] + std::max(0.0, (double)in.progress_weights[i]);
+    if (!(r->cum_w.back() > 0.0)) r->cum_w.clear();
+  }
   r->cov_elems = ctx->cfg.verify ? cov : 0;
   r->trace_elems = (in.flags & ACCEL_REQ_TRACE) ? cov : 0;
   r->clears.assign(in.clear, in.clear + in.n_clear);
@@ -752,15 +765,24 @@ bool fair_weights(accel_ctx* ctx) {
                                   sizeof(uint32_t), cudaMemcpyDeviceToHost, ctx->ctl),
                   "cudaMemcpyAsync(progress)"))
       return false;
+  if (ctx->cuda(cudaEventRecord(ctx->ev_now, ctx->ctl), "cudaEventRecord(now)")) return false;
   if (ctx->cuda(cudaStreamSynchronize(ctx->ctl), "cudaStreamSynchronize(ctl)")) return false;
-  const auto now = std::chrono::steady_clock::now();
   std::vector<double> sig(rs.size(), 0.0);
   int n = 0;
   for (size_t i = 0; i < rs.size(); ++i) {
     Request* r = rs[i];
     r->done_vgs = h[i];
-    const double el = (double)std::chrono::duration_cast<std::chrono::nanoseconds>(now - r->t_submit).count();
-    const double p = std::min(1.0, (double)r->done_vgs / (double)r->vgs_hint);
+    // elapsed device time since the request's first launch was reached on
+    // its stream (not host submission: copies and queueing are not progress)
+    if (!r->ev_start || cudaEventQuery(r->ev_start) != cudaSuccess) continue;
+    float el_ms = 0.f;
+    if (cudaEventElapsedTime(&el_ms, r->ev_start, ctx->ev_now) != cudaSuccess || el_ms <= 0.f) continue;
+    const double el = 1e6 * (double)el_ms;
+    // progress = cost share of the VGs done (progress_weights, in dequeue
+    // order), else their count
+    const double p = r->cum_w.empty()
+        ? std::min(1.0, (double)r->done_vgs / (double)r->vgs_hint)
+        : r->cum_w[std::min<size_t>(r->done_vgs, r->cum_w.size() - 1)] / r->cum_w.back();
     if (p < 0.01 || el < 0.05 * (double)r->iso_ns) continue;  // too early to tell
     sig[i] = el / (p * (double)r->iso_ns);
     ++n;
@@ -888,6 +910,7 @@ void release_request(accel_ctx* ctx, Request* r) {
   if (r->trace) cudaFree(r->trace);
   if (r->ev_arrival) ctx->free_events.push_back(r->ev_arrival);
   if (r->ev_done) ctx->free_events.push_back(r->ev_done);
+  if (r->ev_start) ctx->free_events.push_back(r->ev_start);
   if (r->ev_early) ctx->free_events.push_back(r->ev_early);
   for (cudaEvent_t ev : r->ev_launch) ctx->free_events.push_back(ev);
   for (cudaEvent_t ev : r->ev_topups) ctx->free_events.push_back(ev);
@@ -954,6 +977,7 @@ int accel_init(const accel_config* cfg, accel_ctx** out) {
       return init_fail(e, "cudaStreamCreate");
   if ((e = cudaStreamCreateWithFlags(&ctx->ctl, cudaStreamNonBlocking)) != cudaSuccess)
     return init_fail(e, "cudaStreamCreate");
+  if ((e = cudaEventCreate(&ctx->ev_now)) != cudaSuccess) return init_fail(e, "cudaEventCreate");
   if ((e = cudaEventCreate(&ctx->epoch)) != cudaSuccess) return init_fail(e, "cudaEventCreate");
   if ((e = cudaMalloc(&ctx->pool, (size_t)kPoolSlots * kDescBytes)) != cudaSuccess)
     return init_fail(e, "cudaMalloc(pool)");
@@ -991,6 +1015,7 @@ int accel_finalize(accel_ctx* ctx) {
   for (int t = 0; t < accel_ctx::kTopupStreams; ++t)
     if (ctx->topup[t]) cudaStreamDestroy(ctx->topup[t]);
   if (ctx->ctl) cudaStreamDestroy(ctx->ctl);
+  if (ctx->ev_now) cudaEventDestroy(ctx->ev_now);
   if (ctx->epoch) cudaEventDestroy(ctx->epoch);
   if (ctx->pool) cudaFree(ctx->pool);
   if (ctx->ctl_pool) cudaFree(ctx->ctl_pool);

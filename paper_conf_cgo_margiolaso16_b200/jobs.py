@@ -72,6 +72,8 @@ class Job:
         # FAIR policy: completed VGs / static VGs tracks progress (False for
         # dynamic-total kernels, bfs: they run fewer VGs than their grids)
         self.progress_hint = True
+        # FAIR: relative VG costs in dequeue order (None: every VG counts 1)
+        self.progress_weights: np.ndarray | None = None
 
     # ---- e2e: host buffers ----------------------------------------------
     def pin_host(self) -> None:
@@ -256,6 +258,12 @@ def _lpt_order(cost: np.ndarray, device) -> torch.Tensor:
     return torch.from_numpy(order).to(device)
 
 
+def _weights_in_order(cost: np.ndarray) -> np.ndarray:
+    """FAIR progress weights: the VG costs in the LPT dequeue order."""
+    c = np.asarray(cost, dtype=np.float64)
+    return np.ascontiguousarray(c[np.argsort(-c, kind="stable")], dtype=np.float32)
+
+
 def _cutcp_vg_cost(d: dict, grid) -> np.ndarray:
     """Atoms a cutcp VG streams: the cell rows and trimmed x-ranges its body
     walks (tenants/cutcp.cuh), counted from the cell index."""
@@ -312,7 +320,9 @@ class CutcpJob(Job):
                                          d["ncell_1d"], d["cell"], self.nx, self.ny, self.nz, d["h"],
                                          d["cutoff"], d["excl"], self.v.data_ptr())
         grid = (_cdiv(self.nx, 8), _cdiv(self.ny, 8), _cdiv(self.nz, 8))
-        self.steps = [Step("cutcp", grid, self.args, 1, _lpt_order(_cutcp_vg_cost(d, grid), self.device))]
+        cost = _cutcp_vg_cost(d, grid)
+        self.steps = [Step("cutcp", grid, self.args, 1, _lpt_order(cost, self.device))]
+        self.progress_weights = _weights_in_order(cost)
 
     def result(self):
         return {"v": _np(self.v, np.float32).reshape(self.nz, self.ny, self.nx)}
@@ -342,7 +352,9 @@ class TpacfJob(Job):
                                          p, p + 8 * nb, p + 16 * nb)
         self.clears = [(self.hists, 0)]
         grid = (_cdiv(self.n, 256), 2 * self.S + 1, 1)
-        self.steps = [Step("tpacf", grid, self.args, 1, _lpt_order(_tpacf_vg_cost(self.n, self.S, grid), self.device))]
+        cost = _tpacf_vg_cost(self.n, self.S, grid)
+        self.steps = [Step("tpacf", grid, self.args, 1, _lpt_order(cost, self.device))]
+        self.progress_weights = _weights_in_order(cost)
 
     def result(self):
         h = _np(self.hists, np.uint64).reshape(3, -1)

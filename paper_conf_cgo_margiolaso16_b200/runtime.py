@@ -68,6 +68,10 @@ class Accel:
         if isolated_ms is not None:   # FAIR policy: isolated-time profile per request
             for r, j, ms in zip(reqs, jobs, isolated_ms):
                 r.isolated_ns = int(ms * 1e6) if (ms and j.progress_hint) else 0
+                if r.isolated_ns and j.progress_weights is not None:
+                    w = j.progress_weights   # kept alive by the job until submit returns
+                    r.progress_weights = w.ctypes.data
+                    r.n_progress_weights = len(w)
         # Job buffers (device inputs, tensor maps) were filled on torch's
         # stream; libaccel launches on its own non-blocking streams, which do
         # not order behind it.  Only torch's stream is waited on, never the
