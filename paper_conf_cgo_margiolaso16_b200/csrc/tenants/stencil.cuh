@@ -60,27 +60,36 @@ struct Stencil {
     const int nzt = min(kTZ, nz - z0);
     const int nplanes = nzt + 2;
     const uint32_t sbase = (smem_u32(smem_raw) + 127u) & ~127u;
-    const int rows_total = nz * ny;
-    const int row0 = (z0 - 1) * ny + y0 - 1;            // matrix row of plane 0's first row
-    // my two pieces: e = tid, tid + 256 (< 340); piece e = row e / 34, 16-B column e % 34
+    // my two pieces: e = tid, tid + 256 (< 340); piece e = row e / 34, 16-B column e % 34.
+    // The source address of a piece is fixed per VG up to the plane offset
+    // p * nx * ny, so it is computed once here; per plane only the (uniform)
+    // z range decides whether the piece is read or zero-filled.  Rows y0-1 and
+    // y0+8 outside [0, ny) are zero-filled: they only feed y-face cells, which
+    // copy the input.
     constexpr int kPieces = kRows * (kCols / 4);
     const int e0 = threadIdx.x, e1 = threadIdx.x + kThreads;
     const bool has1 = e1 < kPieces;
     const int rr0 = e0 / (kCols / 4), c0x = x0 - 4 + 4 * (e0 % (kCols / 4));
     const int rr1 = e1 / (kCols / 4), c1x = x0 - 4 + 4 * (e1 % (kCols / 4));
-    const bool colok0 = c0x >= 0 && c0x < nx, colok1 = has1 && c1x >= 0 && c1x < nx;
+    const int ys0 = y0 - 1 + rr0, ys1 = y0 - 1 + rr1;
+    const bool okxy0 = c0x >= 0 && c0x < nx && ys0 >= 0 && ys0 < ny;
+    const bool okxy1 = has1 && c1x >= 0 && c1x < nx && ys1 >= 0 && ys1 < ny;
+    const long long pstr = (long long)nx * ny;
+    // plane p = z0 - 1 + p; offsets of plane 0 (may be negative: only used when valid)
+    const long long off0 = (long long)(z0 - 1) * pstr + (long long)ys0 * nx + c0x;
+    const long long off1 = (long long)(z0 - 1) * pstr + (long long)ys1 * nx + c1x;
     const uint32_t soff0 = 16u * (uint32_t)e0, soff1 = 16u * (uint32_t)e1;
     auto issue = [&](int p) {
       const uint32_t dst = sbase + (uint32_t)(p % kR) * kSlot;
-      const int R0 = row0 + p * ny + rr0;
-      const bool ok0 = colok0 && R0 >= 0 && R0 < rows_total;
-      const float* s0 = ok0 ? in + (size_t)R0 * nx + c0x : in;
+      const int zs = z0 - 1 + p;
+      const bool zok = zs >= 0 && zs < nz;          // uniform
+      const bool ok0 = okxy0 && zok;
+      const float* s0 = ok0 ? in + (off0 + (long long)p * pstr) : in;
       asm volatile("cp.async.cg.shared.global [%0], [%1], 16, %2;" ::"r"(dst + soff0), "l"(s0), "r"(ok0 ? 16 : 0)
                    : "memory");
       if (has1) {
-        const int R1 = row0 + p * ny + rr1;
-        const bool ok1 = colok1 && R1 >= 0 && R1 < rows_total;
-        const float* s1 = ok1 ? in + (size_t)R1 * nx + c1x : in;
+        const bool ok1 = okxy1 && zok;
+        const float* s1 = ok1 ? in + (off1 + (long long)p * pstr) : in;
         asm volatile("cp.async.cg.shared.global [%0], [%1], 16, %2;" ::"r"(dst + soff1), "l"(s1), "r"(ok1 ? 16 : 0)
                      : "memory");
       }
@@ -111,7 +120,6 @@ struct Stencil {
     float4 zm = lds_f4(slot(0) + own);
     float4 cur = lds_f4(slot(1) + own);
     float* po = out + ((size_t)z0 * ny + y) * nx + x0 + 4 * lane;
-    const size_t pstride = (size_t)nx * ny;
 #pragma unroll
     for (int i = 0; i < kTZ; ++i) {
       if (i >= nzt) break;
@@ -133,18 +141,19 @@ struct Stencil {
       if (lane == 0) xl = ev;
       if (lane == 31) xr = ev;
       const int z = z0 + i;
-      const float vx = ((((((zm.x + zp.x) + ym.x) + yp.x) + xl) + cur.y) * c1 - cur.x * c0);
-      const float vy = ((((((zm.y + zp.y) + ym.y) + yp.y) + cur.x) + cur.z) * c1 - cur.y * c0);
-      const float vz = ((((((zm.z + zp.z) + ym.z) + yp.z) + cur.y) + cur.w) * c1 - cur.z * c0);
-      const float vw = ((((((zm.w + zp.w) + ym.w) + yp.w) + cur.z) + xr) * c1 - cur.w * c0);
-      const bool zint = z >= 1 && z <= nz - 2;
-      float4 o;
-      o.x = (zint && mxy[0]) ? vx : cur.x;
-      o.y = (zint && mxy[1]) ? vy : cur.y;
-      o.z = (zint && mxy[2]) ? vz : cur.z;
-      o.w = (zint && mxy[3]) ? vw : cur.w;
+      float4 o = cur;
+      if (z >= 1 && z <= nz - 2) {   // uniform: z-face planes copy the input
+        const float vx = ((((((zm.x + zp.x) + ym.x) + yp.x) + xl) + cur.y) * c1 - cur.x * c0);
+        const float vy = ((((((zm.y + zp.y) + ym.y) + yp.y) + cur.x) + cur.z) * c1 - cur.y * c0);
+        const float vz = ((((((zm.z + zp.z) + ym.z) + yp.z) + cur.y) + cur.w) * c1 - cur.z * c0);
+        const float vw = ((((((zm.w + zp.w) + ym.w) + yp.w) + cur.z) + xr) * c1 - cur.w * c0);
+        if (mxy[0]) o.x = vx;
+        if (mxy[1]) o.y = vy;
+        if (mxy[2]) o.z = vz;
+        if (mxy[3]) o.w = vw;
+      }
       if (active) *reinterpret_cast<float4*>(po) = o;
-      po += pstride;
+      po += pstr;
       zm = cur;
       cur = zp;
     }
