@@ -41,7 +41,17 @@ struct Stencil {
 #endif
   static constexpr int kD = STENCIL_KD;                 // planes in flight beyond z+1
   static constexpr int kR = kD + 2;                     // ring slots
-  static constexpr uint32_t kDynSmem = kR * kSlot + 128;   // + alignment
+#ifndef STENCIL_MBAR
+#define STENCIL_MBAR 0
+#endif
+  // kMbar: per-slot mbarriers instead of one __syncthreads per plane --
+  // "full" completes when all 256 threads' cp.async pieces of the plane landed
+  // (cp.async.mbarrier.arrive.noinc), "empty" when all 8 warps released it, so
+  // warps drift apart by up to a plane instead of meeting at every plane.
+  static constexpr bool kMbar = STENCIL_MBAR != 0;
+  static_assert(!kMbar || kTZ + 2 <= 2 * kR, "a slot is filled at most twice per VG (parities 0, 1)");
+  static constexpr uint32_t kBarBytes = kMbar ? 2 * kR * 8 : 0;
+  static constexpr uint32_t kDynSmem = kR * kSlot + kBarBytes + 128;   // + alignment
 
   // cp.async (LDGSTS, 16 B per copy, L2-only .cg) staging: every thread
   // copies <= 2 of the 340 16-B pieces of a plane tile; out-of-volume pieces are
@@ -60,6 +70,19 @@ struct Stencil {
     const int nzt = min(kTZ, nz - z0);
     const int nplanes = nzt + 2;
     const uint32_t sbase = (smem_u32(smem_raw) + 127u) & ~127u;
+    const uint32_t fullb = sbase + kR * kSlot, emptyb = fullb + kR * 8;   // kMbar only
+    if constexpr (kMbar) {
+      // re-armed per VG: every plane of the previous VG was waited "full" by
+      // every warp (no async arrival pending) and the dispatch barrier closed it
+      if (threadIdx.x == 0) {
+#pragma unroll
+        for (int q = 0; q < kR; ++q) {
+          mbar_init(fullb + 8u * q, kThreads);
+          mbar_init(emptyb + 8u * q, kThreads / 32);
+        }
+      }
+      __syncthreads();
+    }
     // my two pieces: e = tid, tid + 256 (< 340); piece e = row e / 34, 16-B column e % 34.
     // The source address of a piece is fixed per VG up to the plane offset
     // p * nx * ny, so it is computed once here; per plane only the (uniform)
@@ -95,11 +118,22 @@ struct Stencil {
       }
     };
     auto commit = [] { asm volatile("cp.async.commit_group;" ::: "memory"); };
+    auto arrive_full = [&](int p) {   // fires when this thread's copies so far landed
+      asm volatile("cp.async.mbarrier.arrive.noinc.shared::cta.b64 [%0];" ::"r"(fullb + 8u * (uint32_t)(p % kR))
+                   : "memory");
+    };
     // prologue: planes 0 .. kD+1 (one group each, empty groups past the tile)
 #pragma unroll
     for (int p = 0; p < kD + 2; ++p) {
-      if (p < nplanes) issue(p);
-      commit();
+      if constexpr (kMbar) {
+        if (p < nplanes) {
+          issue(p);
+          arrive_full(p);
+        }
+      } else {
+        if (p < nplanes) issue(p);
+        commit();
+      }
     }
     auto slot = [&](int p) { return sbase + (uint32_t)(p % kR) * kSlot; };
 
@@ -114,11 +148,21 @@ struct Stencil {
     const float c0 = a.c0, c1 = a.c1;
     const uint32_t own = 4u * (uint32_t)((warp + 1) * kCols + 4 + 4 * lane);
     const uint32_t edge = 4u * (uint32_t)((warp + 1) * kCols + (lane == 31 ? 4 + kTX : 3));
-    // planes 0 and 1 landed (groups 0, 1 of kD + 2 committed)
-    asm volatile("cp.async.wait_group %0;" ::"n"(kD) : "memory");
-    __syncthreads();
-    float4 zm = lds_f4(slot(0) + own);
-    float4 cur = lds_f4(slot(1) + own);
+    float4 zm, cur;
+    if constexpr (kMbar) {
+      mbar_wait(fullb, 0);
+      mbar_wait(fullb + 8u, 0);
+      zm = lds_f4(slot(0) + own);
+      cur = lds_f4(slot(1) + own);
+      __syncwarp();
+      if (lane == 0) mbar_arrive(emptyb);   // plane 0 released
+    } else {
+      // planes 0 and 1 landed (groups 0, 1 of kD + 2 committed)
+      asm volatile("cp.async.wait_group %0;" ::"n"(kD) : "memory");
+      __syncthreads();
+      zm = lds_f4(slot(0) + own);
+      cur = lds_f4(slot(1) + own);
+    }
     float* po = out + ((size_t)z0 * ny + y) * nx + x0 + 4 * lane;
 #pragma unroll
     for (int i = 0; i < kTZ; ++i) {
@@ -126,11 +170,15 @@ struct Stencil {
       const int pz = i + 1;   // plane pz (= z) is `cur`; plane pz+1 must have landed
       // groups committed: kD + 2 + i; plane pz+1 is group i+2, so at most
       // kD - 1 may still be pending
-      asm volatile("cp.async.wait_group %0;" ::"n"(kD - 1) : "memory");
-      __syncthreads();        // plane pz+1 visible; every thread done with iteration i-1
-      // refill the slot of plane pz-1 (last read in iteration i-1) with plane pz+kD+1
-      if (pz + kD + 1 < nplanes) issue(pz + kD + 1);
-      commit();
+      if constexpr (kMbar) {
+        mbar_wait(fullb + 8u * (uint32_t)((pz + 1) % kR), (uint32_t)(((pz + 1) / kR) & 1));
+      } else {
+        asm volatile("cp.async.wait_group %0;" ::"n"(kD - 1) : "memory");
+        __syncthreads();        // plane pz+1 visible; every thread done with iteration i-1
+        // refill the slot of plane pz-1 (last read in iteration i-1) with plane pz+kD+1
+        if (pz + kD + 1 < nplanes) issue(pz + kD + 1);
+        commit();
+      }
       const uint32_t P = slot(pz);
       const float4 zp = lds_f4(slot(pz + 1) + own);
       const float4 ym = lds_f4(P + own - 4u * kCols);
@@ -151,6 +199,18 @@ struct Stencil {
         if (mxy[1]) o.y = vy;
         if (mxy[2]) o.z = vz;
         if (mxy[3]) o.w = vw;
+      }
+      if constexpr (kMbar) {
+        // plane pz read for the last time (ym, yp, edge): release it; then
+        // refill the slot of plane pz-1 (released by every warp after its
+        // iteration i-1) with plane pz+kD+1
+        __syncwarp();
+        if (lane == 0) mbar_arrive(emptyb + 8u * (uint32_t)(pz % kR));
+        if (pz + kD + 1 < nplanes) {
+          mbar_wait(emptyb + 8u * (uint32_t)((pz - 1) % kR), 0u);
+          issue(pz + kD + 1);
+          arrive_full(pz + kD + 1);
+        }
       }
       if (active) *reinterpret_cast<float4*>(po) = o;
       po += pstr;
