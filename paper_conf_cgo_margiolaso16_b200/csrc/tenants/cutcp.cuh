@@ -35,6 +35,15 @@ struct Cutcp {
   static constexpr int kPts = 4;     // points per thread along z
   static constexpr uint32_t kDynSmem = kTile * sizeof(float4);
 
+  // MUFU.RSQ without the denormal rescaling rsqrtf() wraps around it (4
+  // instructions per in-range pair): r^2 < 2^-126 only occurs for excluded
+  // points (r^2 < e^2), whose output is 0 whatever the sum.
+  static __device__ __forceinline__ float rsqrt_ftz(float x) {
+    float y;
+    asm("rsqrt.approx.ftz.f32 %0, %1;" : "=f"(y) : "f"(x));
+    return y;
+  }
+
   static __device__ __forceinline__ float gap(float lo, float hi, float clo, float chi) {
     // distance between intervals [lo, hi] and [clo, chi]
     return fmaxf(0.f, fmaxf(clo - hi, lo - chi));
@@ -53,12 +62,13 @@ struct Cutcp {
     for (int p = 0; p < kPts; ++p) pz[p] = h * (float)(k0 + p);
     const float c = a.cutoff;
     const float c2 = c * c, e2 = a.excl * a.excl, inv_c2 = 1.0f / c2;
-    float sum[kPts];
-    bool excl[kPts];
+    // excl[p] = "some r^2 < e^2" is kept as the running minimum of r^2 (one
+    // FMNMX per pair instead of a compare, select and byte merge)
+    float sum[kPts], r2min[kPts];
 #pragma unroll
     for (int p = 0; p < kPts; ++p) {
       sum[p] = 0.f;
-      excl[p] = false;
+      r2min[p] = __int_as_float(0x7f800000);   // +inf
     }
     // VG bounding box in Angstrom
     const float bx0 = h * (float)(vb.x * 8), bx1 = h * (float)(vb.x * 8 + 7);
@@ -94,10 +104,10 @@ struct Cutcp {
             for (int p = 0; p < kPts; ++p) {
               const float dz = __fsub_rn(pz[p], at.z);
               const float r2 = __fadd_rn(dxy, __fmul_rn(dz, dz));
-              excl[p] |= r2 < e2;
+              r2min[p] = fminf(r2min[p], r2);
               if (r2 < c2) {
                 const float s = 1.0f - r2 * inv_c2;
-                sum[p] += at.w * rsqrtf(r2) * s * s;
+                sum[p] += at.w * rsqrt_ftz(r2) * s * s;
               }
             }
           }
@@ -108,7 +118,7 @@ struct Cutcp {
 #pragma unroll
       for (int p = 0; p < kPts; ++p) {
         const int k = k0 + p;
-        if (k < (int)a.nz) a.v[((size_t)k * a.ny + j) * a.nx + i] = excl[p] ? 0.f : sum[p];
+        if (k < (int)a.nz) a.v[((size_t)k * a.ny + j) * a.nx + i] = r2min[p] < e2 ? 0.f : sum[p];
       }
     }
   }
