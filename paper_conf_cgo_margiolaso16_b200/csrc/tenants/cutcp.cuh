@@ -21,12 +21,13 @@ struct Cutcp {
   using Args = accel_cutcp_args;
   static constexpr int kThreads = 128;
   static constexpr uint32_t kChunk = 1;
-// 9 resident CTAs/SM caps the body at 56 registers (54 used, no spills; 62
+// 9 resident CTAs/SM caps the body at 56 registers (no spills; 62
 // uncapped).  Registers are cutcp's dominant resource, so its equal share
-// holds 21 % more CTAs: C2 unfairness 2.03-2.09 -> 1.86-1.94 at 1.07x native
-// throughput (1.08x at 8/SM); isolated dispatch overhead 9.5 -> 7.6 %.  At
-// 10/SM (48 registers) C2 reaches U 1.70-1.81 but the isolated persistent
-// run loses 18 % to its tail (profiles/round1_cutcp_regcap.log).
+// holds 21 % more CTAs.  Measured with the branchy loop before the ftz/min
+// change: C2 unfairness 2.03-2.09 -> 1.86-1.94 at 1.07x native throughput,
+// isolated dispatch overhead 9.5 -> 7.6 %; at 10/SM (48 registers) U 1.70-1.81
+// but the isolated persistent run lost 18 % to its tail (DESIGN.md section 6,
+// profiles/round1_cutcp_regcap.log).
 #ifndef CUTCP_MINB
 #define CUTCP_MINB 9
 #endif
