@@ -25,16 +25,15 @@ struct Tpacf {
   static constexpr int kWarps = kThreads / 32;
   static constexpr int kMaxBins = 32;      // nedges + 1 <= 32
   static constexpr int kTile = 256;
-  // [warp][bin][lane] u32 counters + Q tile (3 x 256 floats) + edges (32)
+  // [warp][bin][lane] u32 counters + Q tile (256 float4: x, y, z, pad; one
+  // LDS.128 per pair) + edges (32)
   static constexpr uint32_t kDynSmem =
-      kWarps * kMaxBins * 32 * sizeof(uint32_t) + 3 * kTile * sizeof(float) + 32 * sizeof(float);
+      kWarps * kMaxBins * 32 * sizeof(uint32_t) + kTile * sizeof(float4) + 32 * sizeof(float);
 
   static __device__ __forceinline__ void body(const Args& a, const VirtualBlock& vb, char* smem) {
     uint32_t* hist = reinterpret_cast<uint32_t*>(smem);
-    float* qx = reinterpret_cast<float*>(hist + kWarps * kMaxBins * 32);
-    float* qy = qx + kTile;
-    float* qz = qy + kTile;
-    float* edges = qz + kTile;
+    float4* qt = reinterpret_cast<float4*>(hist + kWarps * kMaxBins * 32);   // 16-B aligned (32 KB of counters)
+    float* edges = reinterpret_cast<float*>(qt + kTile);
     const int t = threadIdx.x, lane = t & 31, warp = t >> 5;
     const uint32_t n = a.npts, S = a.nsets, ne = a.nedges;
     const uint32_t s = vb.y;
@@ -63,27 +62,27 @@ struct Tpacf {
     const float ix = have ? __ldg(P + i) : 0.f, iy = have ? __ldg(P + n + i) : 0.f,
                 iz = have ? __ldg(P + 2 * n + i) : 0.f;
     uint32_t* myh = hist + warp * kMaxBins * 32 + lane;
+    __syncthreads();   // edges staged
+    const float e7 = edges[7], e15 = edges[15], e23 = edges[23];
     const uint32_t j_first_tile = upper ? vb.x * kTile : 0;
     for (uint32_t jt = j_first_tile; jt < n; jt += kTile) {
       __syncthreads();
       const uint32_t jj = jt + t;
-      if (jj < n) {
-        qx[t] = __ldg(Q + jj);
-        qy[t] = __ldg(Q + n + jj);
-        qz[t] = __ldg(Q + 2 * n + jj);
-      }
+      if (jj < n) qt[t] = make_float4(__ldg(Q + jj), __ldg(Q + n + jj), __ldg(Q + 2 * n + jj), 0.f);
       __syncthreads();
       if (!have) continue;
       const uint32_t cnt = min((uint32_t)kTile, n - jt);
       // pairs i < j on the diagonal tile start after i
       const uint32_t q0 = (upper && jt == vb.x * kTile) ? (uint32_t)t + 1 : 0u;
       for (uint32_t q = q0; q < cnt; ++q) {
-        const float d = __fadd_rn(__fadd_rn(__fmul_rn(ix, qx[q]), __fmul_rn(iy, qy[q])),
-                                  __fmul_rn(iz, qz[q]));
-        // bin = #{k : d < edges[k]}; edges descending -> binary search
-        int m = 0;
+        const float4 qv = qt[q];
+        const float d = __fadd_rn(__fadd_rn(__fmul_rn(ix, qv.x), __fmul_rn(iy, qv.y)), __fmul_rn(iz, qv.z));
+        // bin = #{k : d < edges[k]}; edges descending -> binary search, its
+        // first two levels from registers (edges[15], then edges[7] / [23])
+        int m = (e15 > d) ? 16 : 0;
+        if (((m != 0) ? e23 : e7) > d) m += 8;
 #pragma unroll
-        for (int step = 16; step >= 1; step >>= 1)
+        for (int step = 4; step >= 1; step >>= 1)
           if (edges[m + step - 1] > d) m += step;
         myh[m * 32] += 1u;
       }
