@@ -1,4 +1,4 @@
-# final session-4 build (cutcp at 9 CTAs/SM, ftz rsqrt + running-min exclusion): full GPU suite, default bench line, launch list, isolated overheads, C3/C4/f2 mixes
+# final session-4 build (cutcp predicated loop + 56-register cap, tpacf float4 tile): full GPU suite, default bench line, launch list, isolated overheads, C3/C4/f2 mixes
 nvidia-smi --query-gpu=name,clocks.sm,clocks.max.sm --format=csv
 python -m paper_conf_cgo_margiolaso16_b200.build --force > /dev/null 2>&1
 timeout 1500 python -m pytest tests -m gpu -q -x 2>&1 | tail -3
@@ -8,4 +8,3 @@ timeout 600 python scripts/isolated.py stencil histo bfs spmv sgemm mriq cutcp t
 timeout 600 python scripts/mixes.py --config c3 --reps 3 --modes resolve,static --out gpurun_out/c3.json > gpurun_out/c3.log 2>&1; echo "c3 rc=$?"; grep SUMMARY gpurun_out/c3.log | cut -c1-600
 timeout 600 python scripts/mixes.py --config c4 --reps 5 --modes resolve,static --out gpurun_out/c4.json > gpurun_out/c4.log 2>&1; echo "c4 rc=$?"; grep -E "^(native|resolve|static) " gpurun_out/c4.log | cut -c1-160
 timeout 600 python scripts/mixes.py --config f2 --k 4 --n 40 --reps 3 --modes resolve,static --out gpurun_out/f2_k4.json > gpurun_out/f2.log 2>&1; echo "f2 rc=$?"; grep SUMMARY gpurun_out/f2.log | cut -c1-600
-timeout 300 ncu --set full --clock-control none --import-source on -k regex:accel_persistent -s 1 -c 1 -o gpurun_out/s4j_cutcp_static python scripts/profile_one.py cutcp persistent default > /dev/null 2>&1
