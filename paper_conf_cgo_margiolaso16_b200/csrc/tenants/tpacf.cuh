@@ -14,6 +14,10 @@
 #include "../device/dispatch.cuh"
 #include "accel_tenants.h"
 
+#ifndef TPACF_REDS
+#define TPACF_REDS 0
+#endif
+
 namespace accel {
 
 struct Tpacf {
@@ -84,7 +88,13 @@ struct Tpacf {
 #pragma unroll
         for (int step = 4; step >= 1; step >>= 1)
           if (edges[m + step - 1] > d) m += step;
+#if TPACF_REDS
+        // lane-private counter (bank = lane): one RED.ADD on shared memory
+        // instead of load + add + store
+        atomicAdd(myh + m * 32, 1u);
+#else
         myh[m * 32] += 1u;
+#endif
       }
     }
     __syncthreads();
