@@ -15,7 +15,7 @@
 #include "accel_tenants.h"
 
 #ifndef TPACF_REDS
-#define TPACF_REDS 0
+#define TPACF_REDS 1
 #endif
 
 namespace accel {

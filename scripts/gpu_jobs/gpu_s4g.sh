@@ -1,4 +1,4 @@
-# final session-4 build (cutcp predicated loop + 56-register cap, tpacf float4 tile): full GPU suite, default bench line, launch list, isolated overheads, C3/C4/f2 mixes
+# final session-4 build (cutcp predicated loop + 56-register cap, tpacf float4 tile + shared RED counters): full GPU suite, default bench line, launch list, isolated overheads, C3/C4/f2 mixes
 nvidia-smi --query-gpu=name,clocks.sm,clocks.max.sm --format=csv
 python -m paper_conf_cgo_margiolaso16_b200.build --force > /dev/null 2>&1
 timeout 1500 python -m pytest tests -m gpu -q -x 2>&1 | tail -3
