@@ -51,15 +51,8 @@ typedef enum { ACCEL_MODE_NATIVE = 0, ACCEL_MODE_SHARED = 1 } accel_mode;
  * the resources initially allocated").  RESOLVE: quotas are recomputed on every
  * arrival and departure (BASELINE.json north star): shrinking lowers a live
  * quota word read at each dequeue, growing launches extra CTAs.
- * PARTITION: whole SMs are the unit of sharing (the CU split of PAPER.md
- * Fig. 3b): accel_solve_sms gives each active request s_i SMs;
- * its persistent CTAs claim SMs on the device (a per-SM owner word) and run
- * c_i per SM, padded in shared memory so that no other kernel's CTA fits
- * beside them; re-solved on every arrival and departure (an SM is handed over
- * at a VG boundary).  One persistent grid serves all launches of a step.
- * EXPERIMENTAL, disabled: accel_init / accel_set_mode return ACCEL_EINVAL
- * for it unless the environment variable ACCEL_EXPERIMENTAL_PARTITION is set
- * (it halved C2 throughput and one GPU test hung intermittently). */
+ * (Value 2 is retired: an SM-granular PARTITION policy was measured in round
+ * 1 -- half the native throughput on C2 -- and removed.) */
 /* FAIR: RESOLVE whose weights follow the requests' measured slowdowns: the
  * monitor reads each running request's completed VGs every few hundred
  * microseconds, estimates its slowdown so far against its isolated time
@@ -70,7 +63,6 @@ typedef enum { ACCEL_MODE_NATIVE = 0, ACCEL_MODE_SHARED = 1 } accel_mode;
 typedef enum {
   ACCEL_POLICY_STATIC = 0,
   ACCEL_POLICY_RESOLVE = 1,
-  ACCEL_POLICY_PARTITION = 2,
   ACCEL_POLICY_FAIR = 3
 } accel_policy;
 
@@ -125,8 +117,6 @@ typedef struct {
   int32_t regs;               /* regs/thread for the solver; 0 = query attrs   */
   uint32_t chunk;             /* VGs per dequeue (§6.4); 0 = default  */
   uint32_t args_size;         /* sizeof the kernel's argument struct           */
-  const void *partition_fn;   /* host stub of accel_topup<T, PARTITION>; NULL =
-                                 the kernel cannot run under ACCEL_POLICY_PARTITION */
 } accel_kernel_desc;
 
 /* Fill *out with a built-in tenant kernel: "mop", "stencil", "histo", "bfs",
@@ -149,8 +139,6 @@ typedef struct {
   int32_t static_smem;            /* static shared memory of the instance      */
   int32_t occ_persistent;         /* cudaOccupancyMaxActiveBlocksPerMultiprocessor */
   int32_t occ_native;
-  int32_t occ_partition;          /* PARTITION: CTAs per SM c_i (0: none)       */
-  uint32_t partition_smem;        /* PARTITION: padded dynamic smem per CTA     */
 } accel_kernel_info;
 int accel_kernel_info_get(accel_ctx *ctx, int32_t kernel_id, accel_kernel_info *out);
 
@@ -298,13 +286,6 @@ int accel_solve(const accel_caps *caps, const accel_demand *d, int32_t k, uint32
  * SHARED mode enqueues a group's grids in this order and the solver's
  * feasibility model F places them in it.  ACCEL_ENOFIT for an invalid demand. */
 int accel_placement_order(const accel_caps *caps, const accel_demand *d, int32_t k, int32_t *order_out);
-/* SM-granular variant (ACCEL_POLICY_PARTITION; DESIGN.md R-part-1..4): the
- * same closed form + class-symmetric greedy with whole SMs as the one device
- * total.  sms_out[k] = SMs per request (sum <= caps->sms, each <= ceil(G/c));
- * ctas_per_sm_out[k] (may be NULL) = c_i, CTAs of the kernel alone on one SM.
- * ACCEL_ENOFIT if a CTA fits no SM. */
-int accel_solve_sms(const accel_caps *caps, const accel_demand *d, int32_t k, uint32_t *sms_out,
-                    uint32_t *ctas_per_sm_out);
 /* ACCEL_POLICY_FAIR weights (DESIGN.md R-fair-2): from the slowdowns so far
  * slowdown[k] (> 0; <= 0 = not yet known -> the neutral weight 16),
  * weight_out[i] = round(16 * (slowdown_i / g)^2) clamped to [1, 1024], g the

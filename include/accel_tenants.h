@@ -27,7 +27,8 @@ typedef struct {
   uint32_t nconst;
 } accel_mop_args;
 
-/* stencil -- 7-point Jacobi, fp32, A[z][y][x] (x fastest, nx % 4 == 0).
+/* stencil / stencil_x -- 7-point Jacobi, fp32, A[z][y][x] (x fastest).
+ * Kernel "stencil" needs nx % 4 == 0 (16-B rows); "stencil_x" takes any nx.
  * block 256 (8 warps x 32 lanes x 4 x-points), VG tile 128 x 8 x 8 (x,y,z):
  * grid (ceil(nx/128), ceil(ny/8), ceil(nz/8)).  Launch r reads
  * (r == 0 ? a0 : buf[(r-1)&1]) and writes buf[r&1]; after T launches the
@@ -47,8 +48,9 @@ typedef struct {
  * Launch r accumulates into hist[(r&1)*bins + b]; the VG that completes the
  * launch (done[r] reaches the VG count) writes sat[b] = min(hist, 255) and
  * zeroes hist[((r+1)&1)*bins ...] for launch r+1.  The request must clear
- * hist[0..bins) and done[0..launches) first.  bins <= 4096; sample_bytes 1
- * (u8, bins == 256) or 4 (u32). */
+ * hist[0..bins) and done[0..launches) first.  Kernel "histo": bins <= 4096,
+ * sample_bytes 1 (u8, bins == 256) or 4 (u32).  Kernel "histo_wide": bins <=
+ * 16384, sample_bytes 4, per_vg < 65536 (16-bit private counters). */
 typedef struct {
   const void *samples;
   uint32_t n;
@@ -125,7 +127,11 @@ typedef struct {
  * src - hi (exact), for segment 0 (A: src0/hi0/lo0, n0 elements) and
  * segment 1 (B).  block 256, VG = 4096 elements of one segment: VGs
  * [0, ceil(n0/4096)) split A, the next ceil(n1/4096) split B; grid = their
- * sum.  16-B aligned arrays; n1 = 0 for a single array. */
+ * sum.  16-B aligned arrays; n1 = 0 for a single array.  Both sources are
+ * row-major with `cols` (= K) elements per row; hi/lo rows are `ld` >= cols
+ * elements apart (ld = K rounded up to a multiple of 4, so every row starts
+ * 16-B aligned as TMA requires; the pad columns are never read: the tensor
+ * maps' inner extent is cols and TMA zero-fills past it). */
 typedef struct {
   const float *src0;
   float *hi0;
@@ -135,14 +141,15 @@ typedef struct {
   float *hi1;
   float *lo1;
   uint64_t n1;
+  uint32_t cols, ld;
 } accel_sgemm_split_args;
 
 /* sgemm_tc -- C[m][n] = A.B^T on tcgen05 tensor cores, 3xTF32
  * (A_hi.B_hi + A_hi.B_lo + A_lo.B_hi, fp32 accumulation in TMEM).  tmaps =
  * DEVICE pointer to four 128-B CUtensorMaps (A_hi, A_lo, B_hi, B_lo; each a
  * K-major fp32 matrix, box 32 x 128 for A and 32 x 256 for B, 128-B swizzle,
- * see accel_tma_map_2d).  block 128, VG = 128 x 256 tile of C,
- * grid (ceil(n/256), ceil(m/128)).  k % 4 == 0. */
+ * see accel_tma_map_2d; rows 16-B aligned, any k).  block 640, VG = 128 x 256
+ * tile of C, grid (ceil(n/256), ceil(m/128)). */
 typedef struct {
   const void *tmaps;
   float *c;

@@ -162,7 +162,14 @@ def placement_order(ds: Sequence[Demand], caps: Caps = Caps()) -> list[int]:
 
 
 def feasible(ds: Sequence[Demand], n: Sequence[int], caps: Caps = Caps()) -> bool:
-    """Step 3: per-SM feasibility F(n) (R-solver-3).
+    """Step 3: per-SM feasibility F(n) (R-solver-3): the placement below
+    exists."""
+    return placement(ds, n, caps) is not None
+
+
+def placement(ds: Sequence[Demand], n: Sequence[int], caps: Caps = Caps()):
+    """The per-SM placement model behind F(n) (R-solver-3): returns
+    counts[sm][i] = CTAs of request i on SM sm, or None when a CTA fits nowhere.
 
     Kernels in placement order; kernel i's n_i CTAs are dealt round-robin over
     the SMs from a pointer p (carried over between kernels, starting at SM 0),
@@ -198,6 +205,7 @@ def feasible(ds: Sequence[Demand], n: Sequence[int], caps: Caps = Caps()) -> boo
         memo[key] = out
         return out
 
+    counts = [[0] * len(ds) for _ in range(S)]
     p = 0
     for i in placement_order(ds, caps):
         d, left = ds[i], n[i]
@@ -211,12 +219,13 @@ def feasible(ds: Sequence[Demand], n: Sequence[int], caps: Caps = Caps()) -> boo
                     if len(fit) == left:
                         break
             if not fit:
-                return False
+                return None
             for sm, nxt in fit:
                 st[sm] = nxt
+                counts[sm][i] += 1
             left -= len(fit)
             p = (fit[-1][0] + 1) % S
-    return True
+    return counts
 
 
 def dominant_share(d: Demand, n: int, caps: Caps = Caps()) -> Fraction:
@@ -289,79 +298,3 @@ def step_quota(ds: Sequence[Demand], i: int, step: Demand, caps: Caps = Caps()) 
     dj = list(ds)
     dj[i] = step
     return solve(dj, caps)[i]
-
-
-# ---------------------------------------------------------------------------
-# SM-granular partitioning (DESIGN.md R-part-1..4): the same §3 sharing rule
-# with whole SMs as the unit of allocation.  PAPER.md Fig. 3b (lines 441-445)
-# is such a partition -- A's work-groups on CU0/CU1, B's on CU2/CU3 -- and on
-# B200 co-resident CTAs of different kernels share the SM's issue slots under
-# an age-ordered warp scheduler, so only whole SMs give equal shares of every
-# per-SM resource.
-
-def ctas_per_sm(d: Demand, caps: Caps = Caps()) -> int:
-    """R-part-1: c_i = most CTAs of kernel i alone on ONE SM, i.e. the K = 1
-    quota of a one-SM device under the same per-SM model F (pinned against
-    NVIDIA's occupancy calculator through solve())."""
-    check_demand(d, caps)
-    one = Caps(sms=1, thr_per_sm=caps.thr_per_sm, regs_per_sm=caps.regs_per_sm,
-               smem_per_sm=caps.smem_per_sm, ctas_per_sm=caps.ctas_per_sm,
-               smsp_per_sm=caps.smsp_per_sm, max_smem_per_cta=caps.max_smem_per_cta,
-               smem_reserved=caps.smem_reserved, smem_gran=caps.smem_gran,
-               reg_gran=caps.reg_gran, max_regs_per_thread=caps.max_regs_per_thread)
-    c = 0
-    while c < caps.ctas_per_sm and feasible([d], [c + 1], one):
-        c += 1
-    return c
-
-
-def solve_sms(ds: Sequence[Demand], caps: Caps = Caps()) -> tuple[list[int], list[int]]:
-    """SMs s_i (and CTAs per SM c_i) for each active request, arrival order.
-
-    R-part-2, the closed form of PAPER.md lines 525-537 with S SMs as the one
-    device total: s_i = floor(S w_i / W), capped by the SMs the request can
-    use, ceil(G_i / c_i) (R-solver-4), at least 1.
-    R-part-3, if the floors of >= 1 overshoot S (only when K > S or with tiny
-    weights): decrement the class with the largest s_i / w_i (ties: latest
-    class) while it has more than one SM.
-    R-part-4, the greedy of lines 537-542: passes over the classes in order of
-    first arrival, +1 SM per member when every member stays within its cap and
-    the class fits in the free SMs; stop after a pass that accepted nothing.
-    """
-    S = caps.sms
-    c = [ctas_per_sm(d, caps) for d in ds]
-    cap = [ceil_div(d.grid_vgs, ci) for d, ci in zip(ds, c)]
-    W = sum(d.weight for d in ds if d.grid_vgs > 0)
-    s = []
-    for d, ci, gi in zip(ds, c, cap):
-        if d.grid_vgs == 0:
-            s.append(0)
-            continue
-        s.append(max(1, min((S * d.weight) // W, gi)))
-    cls = classes(ds)
-    while sum(s) > S:
-        best = None
-        for ci_, members in enumerate(cls):
-            i = members[0]
-            if s[i] <= 1:
-                continue
-            share = Fraction(s[i], ds[i].weight)
-            if best is None or share >= best[0]:
-                best = (share, ci_)
-        if best is None:
-            break
-        for i in cls[best[1]]:
-            s[i] -= 1
-    while True:
-        accepted = False
-        for members in cls:
-            if any(s[i] + 1 > cap[i] for i in members):
-                continue
-            if sum(s) + len(members) > S:
-                continue
-            for i in members:
-                s[i] += 1
-            accepted = True
-        if not accepted:
-            break
-    return s, c

@@ -23,7 +23,7 @@ ACCEL_ENOTREADY = -7
 ERRORS = {0: "ACCEL_OK", -1: "ACCEL_EINVAL", -2: "ACCEL_ENOFIT", -3: "ACCEL_ECUDA",
           -4: "ACCEL_ESTATE", -5: "ACCEL_ECOVERAGE", -6: "ACCEL_ENOMEM", -7: "ACCEL_ENOTREADY"}
 MODE_NATIVE, MODE_SHARED = 0, 1
-POLICY_STATIC, POLICY_RESOLVE, POLICY_PARTITION, POLICY_FAIR = 0, 1, 2, 3
+POLICY_STATIC, POLICY_RESOLVE, POLICY_FAIR = 0, 1, 3
 ACCEL_ALL = 2**64 - 1
 MAX_TENANTS = 16
 MAX_STEPS = 8
@@ -50,14 +50,12 @@ class accel_kernel_desc(C.Structure):
     _fields_ = [("name", C.c_char_p), ("persistent_fn", vp), ("persistent_resolve_fn", vp), ("native_fn", vp),
                 ("topup_fn", vp),
                 ("block", accel_dim3),
-                ("dyn_smem", u32), ("regs", i32), ("chunk", u32), ("args_size", u32),
-                ("partition_fn", vp)]
+                ("dyn_smem", u32), ("regs", i32), ("chunk", u32), ("args_size", u32)]
 
 
 class accel_kernel_info(C.Structure):
     _fields_ = [("thr", u32), ("regs", u32), ("smem", u32), ("cta", u32), ("num_regs", i32),
-                ("static_smem", i32), ("occ_persistent", i32), ("occ_native", i32),
-                ("occ_partition", i32), ("partition_smem", u32)]
+                ("static_smem", i32), ("occ_persistent", i32), ("occ_native", i32)]
 
 
 class accel_launch(C.Structure):
@@ -145,11 +143,16 @@ class accel_sgemm_args(C.Structure):
 
 class accel_sgemm_split_args(C.Structure):
     _fields_ = [("src0", vp), ("hi0", vp), ("lo0", vp), ("n0", u64),
-                ("src1", vp), ("hi1", vp), ("lo1", vp), ("n1", u64)]
+                ("src1", vp), ("hi1", vp), ("lo1", vp), ("n1", u64), ("cols", u32), ("ld", u32)]
 
 
 class accel_sgemm_tc_args(C.Structure):
     _fields_ = [("tmaps", vp), ("c", vp), ("m", u32), ("n", u32), ("k", u32)]
+
+
+# kernel variants that take the same argument struct
+accel_stencil_x_args = accel_stencil_args
+accel_histo_wide_args = accel_histo_args
 
 
 class accel_mriq_phimag_args(C.Structure):
@@ -165,7 +168,7 @@ EXPORTS = [
     "accel_init", "accel_finalize", "accel_set_mode", "accel_last_error", "accel_builtin_kernel",
     "accel_builtin_count", "accel_builtin_name", "accel_kernel_register", "accel_kernel_info_get",
     "accel_submit", "accel_submit_group", "accel_sync", "accel_epoch", "accel_stats", "accel_release",
-    "accel_tenant_stream", "accel_launch_times", "accel_launch_stats", "accel_vg_trace", "accel_demand_of", "accel_solve", "accel_placement_order", "accel_solve_sms", "accel_fair_weights", "accel_metrics", "accel_overlap", "accel_tma_map_2d",
+    "accel_tenant_stream", "accel_launch_times", "accel_launch_stats", "accel_vg_trace", "accel_demand_of", "accel_solve", "accel_placement_order", "accel_fair_weights", "accel_metrics", "accel_overlap", "accel_tma_map_2d",
 ]
 
 
@@ -204,7 +207,6 @@ def _load() -> C.CDLL:
         "accel_demand_of": (i32, [P(accel_caps), u32, u32, u32, u32, u32, P(accel_demand)]),
         "accel_solve": (i32, [P(accel_caps), P(accel_demand), i32, P(u32)]),
         "accel_placement_order": (i32, [P(accel_caps), P(accel_demand), i32, P(i32)]),
-        "accel_solve_sms": (i32, [P(accel_caps), P(accel_demand), i32, P(u32), P(u32)]),
         "accel_fair_weights": (i32, [P(f64), i32, P(u32)]),
         "accel_metrics": (i32, [P(f64), P(f64), i32, P(accel_mix_metrics)]),
         "accel_overlap": (i32, [P(f64), P(f64), i32, P(f64)]),
@@ -349,16 +351,6 @@ def accel_placement_order(demands: list[accel_demand], caps: accel_caps | None =
     out = (i32 * max(k, 1))()
     check(lib.accel_placement_order(C.byref(caps or accel_caps()), arr, k, out))
     return list(out)[:k]
-
-
-def accel_solve_sms(demands: list[accel_demand], caps: accel_caps | None = None) -> tuple[list[int], list[int]]:
-    """SM-granular partition: (SMs per request, CTAs per SM per request)."""
-    k = len(demands)
-    arr = (accel_demand * max(k, 1))(*demands)
-    sms = (u32 * max(k, 1))()
-    per = (u32 * max(k, 1))()
-    check(lib.accel_solve_sms(C.byref(caps or accel_caps()), arr, k, sms, per))
-    return list(sms)[:k], list(per)[:k]
 
 
 def accel_fair_weights(slowdowns: list[float]) -> list[int]:

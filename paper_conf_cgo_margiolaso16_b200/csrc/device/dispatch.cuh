@@ -20,9 +20,8 @@
 // The body never reads blockIdx/gridDim (the `mop` test catches that), keeps
 // no state across VGs and never waits on another CTA.
 //   accel_persistent<T>: the reduced-grid scheduling kernel (Fig. 8b dyn_sched).
-//   accel_topup<T, P>:   sticky grids that follow a step's launches: RESOLVE
-//                        growth grids (P = false); under PARTITION (P = true)
-//                        every grid of a request (SM claims, see part_claim).
+//   accel_topup<T>:      RESOLVE growth grids: sticky grids that follow a
+//                        step's launches.
 //   accel_native<T>:     the same body on the original grid (Fig. 1a baseline).
 //
 // RESOLVE policy (BASELINE.json north star; not in the paper, whose kernels
@@ -55,10 +54,7 @@ namespace accel {
 struct alignas(128) Ctl {
   // ---- line 0
   uint32_t live;      // live quota (RESOLVE)
-  uint32_t pad0;
-  uint32_t sm_quota;  // PARTITION: SMs the request may own (host-written)
-  uint32_t sm_count;  // PARTITION: SMs it owns (claims - releases); read with sm_quota as one u64
-  uint32_t pad1[28];
+  uint32_t pad1[31];
   // ---- line 1
   uint32_t cur;       // highest request-relative launch index started (one red per launch)
   uint32_t done_vgs;  // FAIR: VGs completed by the request (progress, read by the host monitor)
@@ -89,12 +85,9 @@ struct alignas(128) Desc {
   uint32_t governed;       // RESOLVE: this launch belongs to the request's main
                            // step, whose CTA count the live quota governs (the
                            // other steps keep their own solved grid)
-  uint32_t tok;            // PARTITION: owner token of the request (slot + 1)
-  uint32_t* owner;         // PARTITION: per-SM owner words of the context
-  uint32_t last_step;      // PARTITION: launch of the request's last step
-  uint32_t ctas_per_sm;    // PARTITION: c_i of the step's kernel
+  uint32_t pad_b;
   const uint32_t* order;   // dequeue order (ticket t -> VG order[t]), nullptr = linear
-  uint32_t pad0[8];
+  uint32_t pad0[12];
   // ---- line 1: the software queue head (RUN_TERMINATE when >= total) in the
   // low 32 bits, the admitted CTA count (`alive`, RESOLVE) in the high 32
   unsigned long long qa;
@@ -325,12 +318,6 @@ struct SchedState {
   uint8_t have_nxt, admitted, draining;
   uint8_t over;        // RESOLVE: admitted over the live quota -> leave at the next dequeue
   uint8_t long_vg;     // the last VG ran longer than kLongVgNs
-  uint8_t left;        // PARTITION: the CTA gave up its SM (leaves the sticky loop)
-  // PARTITION, thread 0: this CTA's SM, the request's token, the owner words,
-  // and the views loaded right after the last dequeue (used at the next)
-  uint32_t sm, tok;
-  uint32_t* owner;
-  uint32_t hint_owner, hint_q, hint_c;
   template <bool kSpread>
   __device__ __forceinline__ void set_cur(uint32_t k, uint32_t vg) {
     cur[k].vg = vg;
@@ -348,65 +335,6 @@ struct SchedState {
   }
 };
 
-// ---------------------------------------------------------------------------
-// PARTITION policy (DESIGN.md R-part-*): whole SMs per request.  owner[sm] is
-// 0 (free), tok (owned), tok | kOwnRel (being handed over: claimable by any
-// request under its SM quota, including tok itself) or tok | kOwnClaim (a CTA
-// of tok is claiming it right now).  A request's CTAs are padded in shared
-// memory so that c_i of them fill an SM: no other kernel's CTA fits beside
-// them, which is what makes the partition hold on the hardware.
-constexpr uint32_t kOwnRel = 0x80000000u;
-constexpr uint32_t kOwnClaim = 0x40000000u;
-
-__device__ __forceinline__ unsigned long long ld_relaxed_u64(const void* p) {
-  unsigned long long v;
-  asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
-  return v;
-}
-
-// Thread 0 at CTA start: make this SM the request's (or find it already is).
-// One CTA per SM claims (the kOwnClaim state); the claim takes a ticket on the
-// request's SM count, so at most sm_quota SMs are ever owned.
-__device__ __forceinline__ bool part_claim(uint32_t* owner, Ctl* ctl, uint32_t sm, uint32_t tok) {
-  for (;;) {
-    const uint32_t o = ld_volatile(&owner[sm]);
-    if (o == tok) return true;
-    if (o == (tok | kOwnClaim)) {  // a sibling CTA is claiming this SM
-      __nanosleep(64);
-      continue;
-    }
-    if (o != 0 && !(o & kOwnRel)) return false;  // another request's SM
-    if (atomicCAS(&owner[sm], o, tok | kOwnClaim) != o) continue;
-    const uint32_t cnt = atomicAdd(&ctl->sm_count, 1u);
-    if (cnt < ld_volatile(&ctl->sm_quota)) {
-      atomicExch(&owner[sm], tok);
-      return true;
-    }
-    atomicSub(&ctl->sm_count, 1u);
-    atomicExch(&owner[sm], o);  // at quota: give it back as it was
-    return false;
-  }
-}
-
-// Thread 0 at a dequeue: must this CTA leave its SM?  o_h, q_h, c_h are the
-// owner word and the request's (quota, count) as loaded after the previous
-// dequeue.  Leaves if the SM is no longer the request's; if the request owns
-// more SMs than its quota, the first CTA of an SM to get here marks the SM as
-// handed over (its siblings see the mark at their next dequeue) -- one ticket
-// on the count per SM, so exactly count - quota SMs are released.
-__device__ __forceinline__ bool part_leave(uint32_t* owner, Ctl* ctl, uint32_t sm, uint32_t tok,
-                                           uint32_t o_h, uint32_t q_h, uint32_t c_h) {
-  if (o_h != tok) return true;
-  if (c_h <= q_h) return false;
-  if (atomicCAS(&owner[sm], tok, tok | kOwnRel) != tok) return true;  // a sibling released it
-  const uint32_t cnt = atomicSub(&ctl->sm_count, 1u);
-  if (cnt > ld_volatile(&ctl->sm_quota)) return true;
-  atomicAdd(&ctl->sm_count, 1u);  // enough SMs were released meanwhile: keep it
-  if (atomicCAS(&owner[sm], tok | kOwnRel, tok) == (tok | kOwnRel)) return false;
-  atomicSub(&ctl->sm_count, 1u);  // claimed by another request in between
-  return true;
-}
-
 // One dequeue (Fig. 8b line 26, rt_sched_wgroup): one 64-bit
 // atomicAdd of `chunk` on the queue word, which also returns the admitted
 // count.  Under RESOLVE a CTA first leaves if its last view says the launch
@@ -417,18 +345,17 @@ __device__ __forceinline__ bool part_leave(uint32_t* owner, Ctl* ctl, uint32_t s
 // until retire(), after that VG's results are written.  Returns the raw queue
 // word (kEvicted when the CTA left).
 constexpr unsigned long long kEvicted = ~0ull;
-// RESOLVE slow path of a dequeue: leave the launch (over-admitted, SM handed
-// over) or try to be evicted (alive > live).  Returns true if the CTA left.
+// RESOLVE slow path of a dequeue: leave the launch (over-admitted) or try to
+// be evicted (alive > live).  Returns true if the CTA left.
 // No loops here: a CAS retry loop in this thread-0 branch made the compiler
 // treat the tenant body as possibly divergent and drop the uniform datapath
 // (stencil RESOLVE: 0 vs 38 uniform compares, +6 % instructions executed;
 // ncu source page + cuobjdump), even when moved out of line.
-__device__ __forceinline__ bool try_leave(Desc* d, SchedState* S, bool part_out) {
+__device__ __forceinline__ bool try_leave(Desc* d, SchedState* S) {
   atomicAdd(&d->draining, 1u);
   fence_acq_rel();   // draining visible before alive drops
   bool left = false;
-  if (S->over || part_out) {
-    if (part_out) S->left = 1;
+  if (S->over) {
     atomicAdd(&d->qa, kAliveNeg);
     left = true;
   } else {
@@ -449,11 +376,9 @@ __device__ __forceinline__ bool try_leave(Desc* d, SchedState* S, bool part_out)
   return false;
 }
 
-template <bool kResolve, bool kPart = false>
+template <bool kResolve>
 __device__ __forceinline__ unsigned long long dequeue(Desc* d, SchedState* S) {
-  const bool part_out =
-      kPart && part_leave(S->owner, d->ctl, S->sm, S->tok, S->hint_owner, S->hint_q, S->hint_c);
-  if (kResolve && (part_out || S->over || S->hint_alive > S->hint_live) && try_leave(d, S, part_out))
+  if (kResolve && (S->over || S->hint_alive > S->hint_live) && try_leave(d, S))
     return kEvicted;
   return atomicAdd(&d->qa, (unsigned long long)S->chunk);
 }
@@ -474,7 +399,7 @@ __device__ __forceinline__ void retire(Desc* d, uint32_t cfg, const SchedState* 
 constexpr unsigned long long kLongVgNs = 40000;   // 40 us: ~20 queue round trips
 
 // Serve one launch: admission, dequeue loop, retire.  All threads call it.
-template <class T, bool kResolve, bool kPart = false>
+template <class T, bool kResolve>
 __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, char* smem,
                                       SchedState* S, uint32_t cfg, uint32_t cta_tag) {
   if (threadIdx.x == 0) {    // master work-item: environment init (rt_env_init)
@@ -489,11 +414,6 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     const bool stat = (cfg & kCfgStaticFirst) != 0u;
     if (!kResolve) {
       b = stat ? blockIdx.x * chunk : qa_next(atomicAdd(&d->qa, (unsigned long long)chunk));
-    } else if (kPart && part_leave(S->owner, d->ctl, S->sm, S->tok, S->hint_owner, S->hint_q, S->hint_c)) {
-      // PARTITION: the SM was handed over between two launches: leave unadmitted
-      S->left = 1;
-      S->admitted = 0;
-      b = kTerminate;
     } else {
       // a predecessor launch that was topped up may still be running on its
       // top-up CTAs: this grid's body must wait for it.  The flag load, the
@@ -501,7 +421,7 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
       // launch that was never topped pays no extra round trip
       const uint32_t topped_prev =
           (cfg & kCfgWaitPrev) ? 1u
-          : (!kPart && (cfg & kCfgHasPrev) && !(cfg & kAblNoTop)) ? ld_volatile(&(d - 1)->topped) : 0u;
+          : ((cfg & kCfgHasPrev) && !(cfg & kAblNoTop)) ? ld_volatile(&(d - 1)->topped) : 0u;
       // admission and first dequeue in one atomic; an arrival over the live
       // quota runs the chunk it got and leaves at its next dequeue
       // (a static-first CTA reads the live quota after its first dynamic
@@ -537,7 +457,7 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     if (cfg & kCfgStamps) red_min_u64(&d->t_first, globaltimer());
     const uint32_t launch_idx = d->launch_idx;
     const uint32_t total = vg_total<T>(args, d, launch_idx);
-    // RESOLVE / PARTITION: every CTA publishes the total (the same value: a
+    // RESOLVE: every CTA publishes the total (the same value: a
     // dynamic total is final once the predecessor launch completed).  Top-up
     // CTAs may serve a launch before its main grid is resident -- when they
     // fill the SMs the main grid waits for them -- so completion of a launch
@@ -558,14 +478,14 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     S->order = d->order;
     S->progress = (d->flags & kFlagProgress) ? &d->ctl->done_vgs : nullptr;
     S->spread = has_spread<T>::value ? spread_factor(total) : 0u;
-    S->prefetch_window = 2u * chunk * (kPart ? d->ctas_per_sm * S->hint_q : gridDim.x);
+    S->prefetch_window = 2u * chunk * gridDim.x;
     S->template set_cur<has_spread<T>::value>(0, b);
   }
   __syncthreads();
   // thread 0: the prefetched queue word and live quota stay in registers
   // across the body (a shared-memory store would wait for the atomic)
-  unsigned long long r_v = 0, r_qc = 0;
-  uint32_t r_live = 0, r_own = 0;
+  unsigned long long r_v = 0;
+  uint32_t r_live = 0;
   for (uint32_t k = 0;; k ^= 1u) {
     const SchedState::Cur c = S->cur[k];
     if (c.vg >= S->total) break;                 // RUN_TERMINATE
@@ -577,12 +497,8 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
         // for up to one VG duration.  So kernels whose VGs run long (where
         // that idle time dwarfs one queue round trip) dequeue just in time
         // once fewer than two waves of VGs remain
-        r_v = dequeue<kResolve, kPart>(d, S);
+        r_v = dequeue<kResolve>(d, S);
         if (kResolve) r_live = (d->governed && !(cfg & kAblNoLive)) ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
-        if (kPart) {
-          r_own = ld_relaxed(&S->owner[S->sm]);
-          r_qc = ld_relaxed_u64(&d->ctl->sm_quota);
-        }
         S->have_nxt = 1;
       }
       S->t0 = globaltimer();
@@ -603,17 +519,8 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
         S->template set_cur<has_spread<T>::value>(k ^ 1u, vg + 1);
       } else {                                   // publish the prefetched chunk
         if (!S->have_nxt) {                      // tail: just in time
-          r_v = dequeue<kResolve, kPart>(d, S);
+          r_v = dequeue<kResolve>(d, S);
           if (kResolve) r_live = (d->governed && !(cfg & kAblNoLive)) ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
-          if (kPart) {
-            r_own = ld_relaxed(&S->owner[S->sm]);
-            r_qc = ld_relaxed_u64(&d->ctl->sm_quota);
-          }
-        }
-        if (kPart) {
-          S->hint_owner = r_own;
-          S->hint_q = (uint32_t)r_qc;
-          S->hint_c = (uint32_t)(r_qc >> 32);
         }
         uint32_t nxt = kTerminate;
         if (r_v != kEvicted) {
@@ -647,67 +554,34 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
 // RESOLVE top-up grid: d = first launch of the request step, `sticky` =
 // launches in the step; starts at the request's current launch and follows
 // the step's later launches (each only once its predecessor completed).
-// PARTITION (kPart): the same loop is the request's ONLY kind of grid -- the
-// main grid of every step (c_i x S CTAs on the tenant stream) and the growth
-// grids -- and each CTA first claims its SM (part_claim); a CTA whose SM is
-// not the request's leaves at once, unless the request owns no SM at all
-// (then it serves one chunk as a guest, so a request can never starve).
-template <class T, bool kPart>
+template <class T>
 __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
     accel_topup(const typename T::Args args, Desc* __restrict__ d, uint32_t sticky) {
   extern __shared__ __align__(128) char smem[];
   __shared__ SchedState S;
-  __shared__ uint32_t s_l, s_ok;
+  __shared__ uint32_t s_l;
   if (threadIdx.x == 0) {
     const uint32_t cur = ld_volatile(&d->ctl->cur);
     s_l = cur > d->req_idx ? cur - d->req_idx : 0u;
-    s_ok = 1;
-    S.left = 0;
-    if (kPart) {
-      S.sm = smid();
-      S.tok = d->tok;
-      S.owner = d->owner;
-      const Desc* last = d + (sticky - 1);
-      const uint32_t lt = ld_volatile(&last->total_seen);
-      const bool finished = s_l >= sticky || (lt != kTerminate && qa_next(ld_volatile_u64(&last->qa)) >= lt);
-      bool ok = !finished && part_claim(S.owner, d->ctl, S.sm, S.tok);
-      const unsigned long long qc = ld_relaxed_u64(&d->ctl->sm_quota);
-      S.hint_q = (uint32_t)qc;
-      S.hint_c = (uint32_t)(qc >> 32);
-      // guest: the request owns no SM (all of them are owned by others): run
-      // one chunk here (admitted on a pretended owner view) and leave at the
-      // next dequeue, whose fresh view shows the real owner
-      s_ok = ok || (!finished && S.hint_c == 0);
-      S.hint_owner = s_ok ? S.tok : 0u;
-    }
   }
   __syncthreads();
-  if (!s_ok) return;
   for (uint32_t l = s_l; l < sticky; ++l) {
     Desc* dl = d + l;
     if (threadIdx.x == 0) {
       if (dl->has_prev) wait_complete(dl - 1);  // launch l's inputs are complete
-      if (!kPart) {
-        atomicExch(&dl->topped, 1u);
-        fence_acq_rel();
-      }
+      atomicExch(&dl->topped, 1u);
+      fence_acq_rel();
     }
     __syncthreads();
     // (the predecessor wait above already ran: no kCfgHasPrev)
     const uint32_t cfg = dl->chunk | kCfgResolve | ((dl->flags & kFlagStamps) ? kCfgStamps : 0u);
-    serve<T, true, kPart>(args, dl, smem, &S, cfg, blockIdx.x | (kPart ? 0u : 0x80000000u));
+    serve<T, true>(args, dl, smem, &S, cfg, blockIdx.x | 0x80000000u);
     __syncthreads();
-    if (kPart && S.left) return;
-    // RESOLVE: a top-up CTA that was evicted (shrink) or admitted over the live
-    // quota is surplus: it leaves the request instead of following the later
+    // a top-up CTA that was evicted (shrink) or admitted over the live quota
+    // is surplus: it leaves the request instead of following the later
     // launches (the monitor tops up afresh on a later growth, apply_quota)
-    if (!kPart && (S.over || S.draining)) return;
+    if (S.over || S.draining) return;
   }
-  // the step's last launch is exhausted: free the SM (one CTA per SM wins the
-  // CAS and returns the count); the request's next step claims afresh, so a
-  // step never depends on the SMs an earlier step happened to hold
-  if (kPart && threadIdx.x == 0 && atomicCAS(&S.owner[S.sm], S.tok, 0u) == S.tok)
-    atomicSub(&d->ctl->sm_count, 1u);
 }
 
 // The original kernel: one CTA per VG, hardware block scheduler (Fig. 1a).

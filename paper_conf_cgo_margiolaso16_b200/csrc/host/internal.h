@@ -18,7 +18,6 @@ struct InitStep {
   uint32_t gx, gy, gz;
   uint32_t chunk;
   uint32_t cov_offset; // coverage offset of the step's first launch
-  uint32_t ctas_per_sm; // PARTITION: c_i of the step's kernel (0 otherwise)
   const uint32_t* order; // dequeue order (nullptr: linear)
   uint64_t qa0;          // initial queue word (alive << 32 | next): main grids with
                          // static first chunks start at grid*chunk (alive = grid
@@ -35,16 +34,12 @@ struct InitParams {
   uint32_t flags;
   uint32_t n_steps;
   InitStep steps[ACCEL_MAX_STEPS];
-  uint32_t* owner;        // PARTITION: the context's per-SM owner words (else nullptr)
-  uint32_t tok;           // PARTITION: the request's owner token
-  uint32_t sm_quota_init; // PARTITION: initial SM quota
 };
 
 // Fill the descriptors of one request on `s` (one tiny kernel).
 cudaError_t launch_desc_init(const InitParams& p, uint32_t n_desc, cudaStream_t s);
 // RESOLVE: wait (1 thread) until the request's last launch and its top-ups completed.
-// PARTITION: then release the SMs the request still owns (nsm owner words).
-cudaError_t launch_join(const Desc* last, uint32_t nsm, cudaStream_t s);
+cudaError_t launch_join(const Desc* last, cudaStream_t s);
 constexpr size_t kDescBytes = 384;
 constexpr size_t kCtlBytes = 256;
 

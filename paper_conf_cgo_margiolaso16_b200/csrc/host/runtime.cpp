@@ -36,7 +36,6 @@ using accel::kDescBytes;
 
 constexpr uint32_t kPoolSlots = 16384;      // 4 MiB of descriptors
 constexpr uint32_t kFlagStamps = 1u, kFlagAlive = 2u;  // dispatch.cuh
-constexpr uint32_t kOwnerWords = 1024;     // %smid < 1024 (ids need not be contiguous)
 constexpr uint32_t kFlagProgress = 4u;     // dispatch.cuh: count completed VGs in Ctl::done_vgs
 constexpr int kFairPeriodUs = 150;         // FAIR: feedback period of the monitor
 constexpr double kFairW0 = 16.0;           // FAIR: neutral weight
@@ -50,9 +49,6 @@ struct Kernel {
   const void* prfn;  // accel_persistent<T, RESOLVE>
   const void* nfn;
   const void* tfn;
-  const void* partfn;   // accel_topup<T, PARTITION> (nullptr: not partitionable)
-  int occ_part = 0;     // PARTITION: CTAs per SM (c_i) of partfn
-  uint32_t part_smem = 0;  // PARTITION: dynamic smem padded so c_i CTAs fill the SM
   dim3 block;
   uint32_t dyn_smem;
   uint32_t chunk;
@@ -86,6 +82,10 @@ struct Request {
   std::vector<accel_clear> clears;
   std::vector<accel_copy> h2d, d2h;
   cudaEvent_t ev_arrival = nullptr, ev_done = nullptr;
+  // recorded on the tenant stream right after the descriptor init: everything
+  // that touches the request's descriptors or control block from another
+  // stream (growth grids, live-quota writes, the early main grid) waits on it
+  cudaEvent_t ev_init = nullptr;
   std::vector<cudaEvent_t> ev_launch;  // ACCEL_REQ_LAUNCH_EVENTS: n_desc + 1
   // RESOLVE: one event after every top-up grid.  The request's descriptors
   // may only be released (and reused) once its sticky top-up CTAs retired.
@@ -103,15 +103,12 @@ struct Request {
   cudaEvent_t ev_early = nullptr;  // recorded after that launch (the main stream waits for it)
   uint32_t live = 0;         // RESOLVE: current live quota of the main step
   uint32_t provisioned = 0;  // RESOLVE: main-grid CTAs + sticky top-up CTAs
-  bool part = false;         // PARTITION request
   uint64_t iso_ns = 0;       // FAIR: isolated-time hint (0: none)
   uint64_t vgs_hint = 0;     // FAIR: VGs the request runs
   std::vector<double> cum_w; // FAIR: prefix sums of the progress weights (empty: count VGs)
   cudaEvent_t ev_start = nullptr;  // FAIR: before the first launch (device-time elapsed)
   std::chrono::steady_clock::time_point t_submit;
   uint32_t done_vgs = 0;     // FAIR: last progress read
-  uint32_t sms = 0;          // PARTITION: current SM quota
-  uint32_t sms_provisioned = 0;  // PARTITION: SMs' worth of CTAs launched for the main step
   bool done = false;
   bool departed_seen = false;  // monitor already re-solved for this departure
   bool fetched = false;
@@ -146,11 +143,9 @@ struct DescHost {
   uint64_t ctl, coverage;
   uint32_t has_prev, pad_a;
   uint64_t trace;
-  uint32_t governed, tok;
-  uint64_t owner;
-  uint32_t last_step, ctas_per_sm;
+  uint32_t governed, pad_b;
   uint64_t order;
-  uint32_t pad0[8];
+  uint32_t pad0[12];
   // line 1
   unsigned long long qa;  // alive << 32 | next
   uint32_t pad1[30];
@@ -196,7 +191,6 @@ struct accel_ctx {
   bool epoch_set = false;
   unsigned char* pool = nullptr;
   unsigned char* ctl_pool = nullptr;      // accel::Ctl per descriptor slot
-  uint32_t* owner = nullptr;              // PARTITION: per-SM owner words (kOwnerWords)
   uint32_t* pinned_ring = nullptr;        // staging for live-quota writes
   uint32_t ring_pos = 0;
   std::thread monitor;
@@ -319,8 +313,8 @@ int fetch_result(accel_ctx* ctx, Request* r) {
 
 // Enqueue of one request, in three parts so that a group's requests can be
 // interleaved (enqueue_group): begin = arrival event, clears, copies,
-// descriptor init; then its launch units (one per launch; one per step under
-// PARTITION) in order; end = join, copies back, done event.
+// descriptor init; then its launch units (one per launch) in order; end =
+// join, copies back, done event.
 int enqueue_begin(accel_ctx* ctx, Request* r) {
   const bool shared = r->mode == ACCEL_MODE_SHARED;
   cudaStream_t s = ctx->main[r->tenant];
@@ -333,13 +327,9 @@ int enqueue_begin(accel_ctx* ctx, Request* r) {
   if (r->trace) CK(ctx, cudaMemsetAsync(r->trace, 0, r->trace_elems * sizeof(accel_vg_record), s));
   InitParams p{};
   p.d = ctx->desc_ptr(r->slot);
-  const bool part = shared && r->part;
-  const bool resolve = shared && (is_resolve(ctx->cfg.policy) || part);
+  const bool resolve = shared && is_resolve(ctx->cfg.policy);
   p.ctl = resolve ? ctx->ctl_ptr(r->slot) : nullptr;
-  p.live_init = part ? 0xffffffffu : r->steps[r->main_step].quota;
-  p.owner = part ? ctx->owner : nullptr;
-  p.tok = r->slot + 1;
-  p.sm_quota_init = r->sms;
+  p.live_init = r->steps[r->main_step].quota;
   p.main_step = (uint32_t)r->main_step;
   p.coverage = r->cov;
   p.trace = r->trace;
@@ -349,16 +339,19 @@ int enqueue_begin(accel_ctx* ctx, Request* r) {
   for (size_t j = 0; j < r->steps.size(); ++j) {
     const Step& st = r->steps[j];
     const Kernel& k = ctx->kernels[st.kid];
-    // main grids (SHARED, not PARTITION) take static first chunks: the queue
-    // head starts past them and, under RESOLVE, every main-grid CTA is admitted
-    const uint64_t qa0 = (shared && !part)
+    // main grids (SHARED) take static first chunks: the queue head starts
+    // past them and, under RESOLVE, every main-grid CTA is admitted
+    const uint64_t qa0 = shared
         ? ((resolve ? (uint64_t)st.quota << 32 : 0ull) | ((uint64_t)st.quota * k.chunk))
         : 0ull;
     p.steps[j] = accel::InitStep{st.first, st.repeat, st.total, st.grid.x, st.grid.y, st.grid.z,
-                                 k.chunk, (uint32_t)st.cov_offset, part ? (uint32_t)k.occ_part : 0u,
-                                 shared ? st.order : nullptr, qa0};
+                                 k.chunk, (uint32_t)st.cov_offset, shared ? st.order : nullptr, qa0};
   }
   CK(ctx, accel::launch_desc_init(p, r->n_desc, s));
+  if (resolve) {
+    CK(ctx, ctx->get_event(&r->ev_init));
+    CK(ctx, cudaEventRecord(r->ev_init, s));
+  }
   if (shared && ctx->cfg.policy == ACCEL_POLICY_FAIR && r->iso_ns) {
     CK(ctx, ctx->get_event(&r->ev_start));
     CK(ctx, cudaEventRecord(r->ev_start, s));
@@ -380,7 +373,7 @@ int enqueue_begin(accel_ctx* ctx, Request* r) {
   // to run).
   r->early_main = false;
   const size_t ms = (size_t)r->main_step;
-  if (shared && !part && resolve && ms > 0 && ms + 1 == r->steps.size() && r->steps[ms].repeat == 1 &&
+  if (shared && resolve && ms > 0 && ms + 1 == r->steps.size() && r->steps[ms].repeat == 1 &&
       // the early grids' CTAs wait on the device while holding (up to) an SM
       // each: together they may hold at most half the device, so the earlier
       // steps and every co-runner always have SMs to make progress on (two
@@ -396,12 +389,8 @@ int enqueue_begin(accel_ctx* ctx, Request* r) {
       r->early_main = true;
       r->early_sms = st.quota;
       ctx->early_sms += st.quota;
-      cudaEvent_t ev_init;
-      CK(ctx, ctx->get_event(&ev_init));
-      CK(ctx, cudaEventRecord(ev_init, s));            // descriptors initialised
       cudaStream_t es = ctx->pick_topup_stream();
-      CK(ctx, cudaStreamWaitEvent(es, ev_init, 0));
-      ctx->free_events.push_back(ev_init);             // reusable once recorded + waited on
+      CK(ctx, cudaStreamWaitEvent(es, r->ev_init, 0));  // descriptors initialised
       accel::Desc* d = ctx->desc_ptr(r->slot + st.first);
       // kCfgResolve | kCfgStamps | kCfgHasPrev | kCfgStaticFirst | kCfgWaitPrev
       uint32_t cfg = (k.chunk & 0xffffu) | (1u << 16) | (1u << 17) | (1u << 18) | (1u << 19) | (1u << 20) | ctx->ablate;
@@ -417,8 +406,7 @@ int enqueue_begin(accel_ctx* ctx, Request* r) {
 // Enqueue the request's next launch unit; *more = false once all are enqueued.
 int enqueue_next(accel_ctx* ctx, Request* r, bool* more) {
   const bool shared = r->mode == ACCEL_MODE_SHARED;
-  const bool part = shared && r->part;
-  const bool resolve = shared && (is_resolve(ctx->cfg.policy) || part);
+  const bool resolve = shared && is_resolve(ctx->cfg.policy);
   const bool lev = (r->flags & ACCEL_REQ_LAUNCH_EVENTS) != 0;
   cudaStream_t s = ctx->main[r->tenant];
   const size_t n_units = r->early_main ? (size_t)r->main_step : r->steps.size();
@@ -430,18 +418,7 @@ int enqueue_next(accel_ctx* ctx, Request* r, bool* more) {
   const Kernel& k = ctx->kernels[st.kid];
   const uint32_t li = r->enq_li;
   if (lev) CK(ctx, cudaEventRecord(r->ev_launch[li], s));
-  if (part) {
-    // PARTITION: one sticky grid per step serves all its launches; c_i CTAs
-    // for every SM of the device, so whichever SMs the request gets are
-    // filled (the CTAs on SMs it does not get leave at once)
-    accel::Desc* d = ctx->desc_ptr(r->slot + st.first);
-    uint32_t sticky = st.repeat;
-    void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &sticky};
-    CK(ctx, cudaLaunchKernel(k.partfn, dim3((uint32_t)k.occ_part * (uint32_t)ctx->caps.sms, 1, 1), k.block,
-                             params, k.part_smem, s));
-    r->enq_li += st.repeat;
-    r->enq_step += 1;
-  } else {
+  {
     const uint32_t l = r->enq_launch;
     accel::Desc* d = ctx->desc_ptr(r->slot + st.first + l);
     // accel_persistent cfg word (dispatch.cuh): chunk | kCfgResolve | kCfgStamps
@@ -463,8 +440,7 @@ int enqueue_next(accel_ctx* ctx, Request* r, bool* more) {
 
 int enqueue_end(accel_ctx* ctx, Request* r) {
   const bool shared = r->mode == ACCEL_MODE_SHARED;
-  const bool part = shared && r->part;
-  const bool resolve = shared && (is_resolve(ctx->cfg.policy) || part);
+  const bool resolve = shared && is_resolve(ctx->cfg.policy);
   cudaStream_t s = ctx->main[r->tenant];
   if (r->early_main) {
     // launch-time stamps: the early grid's work starts once the earlier
@@ -474,7 +450,7 @@ int enqueue_end(accel_ctx* ctx, Request* r) {
     r->enq_li = r->n_desc;   // the early launch was the last one
   }
   if (r->flags & ACCEL_REQ_LAUNCH_EVENTS) CK(ctx, cudaEventRecord(r->ev_launch[r->enq_li], s));
-  if (resolve) CK(ctx, accel::launch_join(ctx->desc_ptr(r->slot + r->n_desc - 1), part ? kOwnerWords : 0u, s));
+  if (resolve) CK(ctx, accel::launch_join(ctx->desc_ptr(r->slot + r->n_desc - 1), s));
   for (const accel_copy& c : r->d2h) CK(ctx, cudaMemcpyAsync(c.dst, c.src, c.bytes, cudaMemcpyDeviceToHost, s));
   CK(ctx, cudaEventRecord(r->ev_done, s));
   return ACCEL_OK;
@@ -523,7 +499,6 @@ int build_request(accel_ctx* ctx, const accel_request& in, std::unique_ptr<Reque
   r->flags = in.flags;
   r->weight = in.weight ? in.weight : 1;
   r->mode = ctx->cfg.mode;
-  r->part = ctx->cfg.mode == ACCEL_MODE_SHARED && ctx->cfg.policy == ACCEL_POLICY_PARTITION;
   r->iso_ns = in.isolated_ns;
   r->t_submit = std::chrono::steady_clock::now();
   if (ctx->cfg.policy == ACCEL_POLICY_FAIR) r->weight = (uint32_t)kFairW0 * r->weight;  // neutral = W0
@@ -537,8 +512,6 @@ int build_request(accel_ctx* ctx, const accel_request& in, std::unique_ptr<Reque
     const Kernel& k = ctx->kernels[L.kernel_id];
     if (L.args_size != k.args_size || !L.args) return ctx->fail(ACCEL_EINVAL, "args_size mismatch for " + k.name);
     if (L.repeat < 1) return ctx->fail(ACCEL_EINVAL, "repeat < 1");
-    if (r->part && (!k.partfn || k.occ_part < 1))
-      return ctx->fail(ACCEL_EINVAL, k.name + " has no PARTITION instantiation");
     const uint64_t total = (uint64_t)L.grid.x * L.grid.y * L.grid.z;
     if (total == 0 || total >= 0x7fffffffull || L.grid.y > 65535 || L.grid.z > 65535)
       return ctx->fail(ACCEL_EINVAL, "bad grid");
@@ -591,10 +564,14 @@ int apply_quota(accel_ctx* ctx, Request* r, uint32_t q) {
   if (debug_on())
     std::fprintf(stderr, "[accel] resolve req %llu tenant %d live %u -> %u (provisioned %u)\n",
                  (unsigned long long)r->id, r->tenant, r->live, q, r->provisioned);
-  if (q == r->live) return ACCEL_OK;
+  if (q == r->live || r->ev_init == nullptr) return ACCEL_OK;
   if (cudaEventQuery(r->ev_done) == cudaSuccess) return ACCEL_OK;  // finished: nothing to grow
   uint32_t* h = ctx->pinned_ring + (ctx->ring_pos++ % kRing);
   *h = q;
+  // both the live-quota write and a growth grid must follow the request's
+  // descriptor init (which writes live_init and resets the queue words): a
+  // re-solve may come while the tenant stream is still copying its inputs
+  CK(ctx, cudaStreamWaitEvent(ctx->ctl, r->ev_init, 0));
   CK(ctx, cudaMemcpyAsync(ctx->ctl_pool + (size_t)r->slot * kCtlBytes /* Ctl::live */, h, sizeof(uint32_t), cudaMemcpyHostToDevice, ctx->ctl));
   // (no growth grids for an early main step: they would wait beside it for
   // the earlier steps and could hold the SMs those need)
@@ -605,6 +582,7 @@ int apply_quota(accel_ctx* ctx, Request* r, uint32_t q) {
     uint32_t sticky = st.repeat;
     void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &sticky};
     cudaStream_t ts = ctx->pick_topup_stream();
+    CK(ctx, cudaStreamWaitEvent(ts, r->ev_init, 0));
     CK(ctx, cudaLaunchKernel(k.tfn, dim3(q - r->provisioned, 1, 1), k.block, params, k.dyn_smem, ts));
     cudaEvent_t ev;
     CK(ctx, ctx->get_event(&ev));
@@ -621,70 +599,6 @@ int apply_quota(accel_ctx* ctx, Request* r, uint32_t q) {
   return ACCEL_OK;
 }
 
-// PARTITION: set a running request's SM quota (copy engine).  Shrinking takes
-// effect at its CTAs' next dequeues (part_leave); growing relies on the main
-// grid's CTAs still waiting for an SM and, as insurance, adds a growth grid of
-// c_i CTAs per extra SM (its CTAs that find no SM to claim leave at once).
-int apply_sms(accel_ctx* ctx, Request* r, uint32_t sms) {
-  if (debug_on())
-    std::fprintf(stderr, "[accel] partition req %llu tenant %d sms %u -> %u\n", (unsigned long long)r->id,
-                 r->tenant, r->sms, sms);
-  if (sms == r->sms) return ACCEL_OK;
-  if (cudaEventQuery(r->ev_done) == cudaSuccess) return ACCEL_OK;
-  uint32_t* h = ctx->pinned_ring + (ctx->ring_pos++ % kRing);
-  *h = sms;
-  CK(ctx, cudaMemcpyAsync(ctx->ctl_pool + (size_t)r->slot * kCtlBytes + 8 /* Ctl::sm_quota */, h,
-                          sizeof(uint32_t), cudaMemcpyHostToDevice, ctx->ctl));
-  if (sms > r->sms_provisioned) {
-    const Step& st = r->steps[r->main_step];
-    const Kernel& k = ctx->kernels[st.kid];
-    accel::Desc* d = ctx->desc_ptr(r->slot + st.first);
-    uint32_t sticky = st.repeat;
-    void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &sticky};
-    cudaStream_t ts = ctx->pick_topup_stream();
-    CK(ctx, cudaLaunchKernel(k.partfn, dim3((sms - r->sms_provisioned) * (uint32_t)k.occ_part, 1, 1), k.block,
-                             params, k.part_smem, ts));
-    cudaEvent_t ev;
-    CK(ctx, ctx->get_event(&ev));
-    r->ev_topups.push_back(ev);
-    CK(ctx, cudaEventRecord(ev, ts));
-    r->sms_provisioned = sms;
-  }
-  const uint32_t c = (uint32_t)ctx->kernels[r->steps[r->main_step].kid].occ_part;
-  r->sms = sms;
-  r->live = sms * c;
-  r->resolves += 1;
-  r->quota_min = std::min(r->quota_min, sms * c);
-  r->quota_max = std::max(r->quota_max, sms * c);
-  return ACCEL_OK;
-}
-
-int assign_sms(accel_ctx* ctx, const std::vector<Request*>& order, size_t first_new) {
-  std::vector<accel_demand> ds(order.size());
-  for (size_t i = 0; i < order.size(); ++i) {
-    Request* r = order[i];
-    int rc = demand_for(ctx, r->steps[r->main_step], r->weight, &ds[i]);
-    if (rc) return ctx->fail(rc, "kernel does not fit on an SM");
-  }
-  std::vector<uint32_t> sms(order.size()), per(order.size());
-  int rc = accel_solve_sms(&ctx->caps, ds.data(), (int32_t)ds.size(), sms.data(), per.data());
-  if (rc) return ctx->fail(rc, "accel_solve_sms failed");
-  ctx->monitor_solves += 1;
-  for (size_t i = 0; i < first_new; ++i) {
-    rc = apply_sms(ctx, order[i], sms[i]);
-    if (rc) return rc;
-  }
-  for (size_t i = first_new; i < order.size(); ++i) {
-    Request* r = order[i];
-    const uint32_t c = (uint32_t)ctx->kernels[r->steps[r->main_step].kid].occ_part;
-    for (Step& st : r->steps) st.quota = sms[i] * (uint32_t)ctx->kernels[st.kid].occ_part;
-    r->sms = r->sms_provisioned = sms[i];
-    r->quota_initial = r->quota_min = r->quota_max = sms[i] * c;
-    r->live = r->provisioned = sms[i] * c;
-  }
-  return ACCEL_OK;
-}
-
 // Solve over the active requests (arrival order) + the new ones.  STATIC:
 // running requests keep their quota and only the new
 // ones are assigned.  RESOLVE: every active request gets its new quota.
@@ -698,7 +612,6 @@ int assign_quotas(accel_ctx* ctx, std::vector<std::unique_ptr<Request>>& fresh) 
   }
   for (auto& r : fresh) order.push_back(r.get());
   if (order.empty()) return ACCEL_OK;
-  if (ctx->cfg.policy == ACCEL_POLICY_PARTITION) return assign_sms(ctx, order, order.size() - fresh.size());
   std::vector<accel_demand> ds(order.size());
   for (size_t i = 0; i < order.size(); ++i) {
     Request* r = order[i];
@@ -912,6 +825,7 @@ void release_request(accel_ctx* ctx, Request* r) {
   if (r->ev_done) ctx->free_events.push_back(r->ev_done);
   if (r->ev_start) ctx->free_events.push_back(r->ev_start);
   if (r->ev_early) ctx->free_events.push_back(r->ev_early);
+  if (r->ev_init) ctx->free_events.push_back(r->ev_init);
   for (cudaEvent_t ev : r->ev_launch) ctx->free_events.push_back(ev);
   for (cudaEvent_t ev : r->ev_topups) ctx->free_events.push_back(ev);
 }
@@ -941,19 +855,15 @@ const char* accel_last_error(const accel_ctx* ctx) {
   return ctx ? ctx->err.c_str() : g_init_error.c_str();
 }
 
-// PARTITION is experimental and off unless ACCEL_EXPERIMENTAL_PARTITION is
-// set: it lost half the native throughput on C2 and one of its single-tenant
-// GPU tests hung intermittently
 bool policy_enabled(int32_t policy) {
-  if (policy == ACCEL_POLICY_STATIC || policy == ACCEL_POLICY_RESOLVE || policy == ACCEL_POLICY_FAIR) return true;
-  return policy == ACCEL_POLICY_PARTITION && std::getenv("ACCEL_EXPERIMENTAL_PARTITION") != nullptr;
+  return policy == ACCEL_POLICY_STATIC || policy == ACCEL_POLICY_RESOLVE || policy == ACCEL_POLICY_FAIR;
 }
 
 int accel_init(const accel_config* cfg, accel_ctx** out) {
   if (!cfg || !out) return ACCEL_EINVAL;
   if (cfg->mode != ACCEL_MODE_NATIVE && cfg->mode != ACCEL_MODE_SHARED) return ACCEL_EINVAL;
   if (!policy_enabled(cfg->policy)) {
-    g_init_error = "bad or disabled policy (PARTITION needs ACCEL_EXPERIMENTAL_PARTITION=1)";
+    g_init_error = "bad policy";
     return ACCEL_EINVAL;
   }
   auto ctx = std::make_unique<accel_ctx>();
@@ -983,10 +893,6 @@ int accel_init(const accel_config* cfg, accel_ctx** out) {
     return init_fail(e, "cudaMalloc(pool)");
   if ((e = cudaMalloc(&ctx->ctl_pool, (size_t)kPoolSlots * kCtlBytes)) != cudaSuccess)
     return init_fail(e, "cudaMalloc(ctl)");
-  if ((e = cudaMalloc(&ctx->owner, kOwnerWords * sizeof(uint32_t))) != cudaSuccess)
-    return init_fail(e, "cudaMalloc(owner)");
-  if ((e = cudaMemset(ctx->owner, 0, kOwnerWords * sizeof(uint32_t))) != cudaSuccess)
-    return init_fail(e, "cudaMemset(owner)");
   if ((e = cudaHostAlloc(reinterpret_cast<void**>(&ctx->pinned_ring), kRing * sizeof(uint32_t),
                          cudaHostAllocDefault)) != cudaSuccess)
     return init_fail(e, "cudaHostAlloc(ring)");
@@ -1019,7 +925,6 @@ int accel_finalize(accel_ctx* ctx) {
   if (ctx->epoch) cudaEventDestroy(ctx->epoch);
   if (ctx->pool) cudaFree(ctx->pool);
   if (ctx->ctl_pool) cudaFree(ctx->ctl_pool);
-  if (ctx->owner) cudaFree(ctx->owner);
   if (ctx->pinned_ring) cudaFreeHost(ctx->pinned_ring);
   delete ctx;
   return ACCEL_OK;
@@ -1031,7 +936,7 @@ int accel_set_mode(accel_ctx* ctx, int32_t mode, int32_t policy) {
   if (ctx->poisoned) return ACCEL_ESTATE;
   if (mode != ACCEL_MODE_NATIVE && mode != ACCEL_MODE_SHARED) return ctx->fail(ACCEL_EINVAL, "bad mode");
   if (!policy_enabled(policy))
-    return ctx->fail(ACCEL_EINVAL, "bad or disabled policy (PARTITION needs ACCEL_EXPERIMENTAL_PARTITION=1)");
+    return ctx->fail(ACCEL_EINVAL, "bad policy");
   for (auto& kv : ctx->reqs) {
     int rc = refresh_done(ctx, kv.second.get());
     if (rc) return rc;
@@ -1053,7 +958,6 @@ int accel_kernel_register(accel_ctx* ctx, const accel_kernel_desc* d, int32_t* k
   k.prfn = d->persistent_resolve_fn ? d->persistent_resolve_fn : d->persistent_fn;
   k.nfn = d->native_fn;
   k.tfn = d->topup_fn ? d->topup_fn : d->persistent_fn;
-  k.partfn = d->partition_fn;
   k.block = dim3(d->block.x, d->block.y ? d->block.y : 1, d->block.z ? d->block.z : 1);
   k.dyn_smem = d->dyn_smem;
   k.chunk = d->chunk ? d->chunk : 1;
@@ -1075,39 +979,6 @@ int accel_kernel_register(accel_ctx* ctx, const accel_kernel_desc* d, int32_t* k
   }
   CK(ctx, cudaOccupancyMaxActiveBlocksPerMultiprocessor(&k.occ_p, k.pfn, (int)k.threads(), k.dyn_smem));
   CK(ctx, cudaOccupancyMaxActiveBlocksPerMultiprocessor(&k.occ_n, k.nfn, (int)k.threads(), k.dyn_smem));
-  if (k.partfn) {
-    // PARTITION: c_i CTAs alone on an SM, then pad the dynamic shared memory so
-    // that exactly c_i of them take all of it (1 KiB reserved per CTA, 128-B
-    // granules): no CTA of another kernel fits on an SM the request holds
-    CK(ctx, cudaFuncSetAttribute(k.partfn, cudaFuncAttributePreferredSharedMemoryCarveout, 100));
-    if (k.dyn_smem > 48 * 1024)
-      CK(ctx, cudaFuncSetAttribute(k.partfn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)k.dyn_smem));
-    cudaFuncAttributes pa;
-    CK(ctx, cudaFuncGetAttributes(&pa, k.partfn));
-    CK(ctx, cudaOccupancyMaxActiveBlocksPerMultiprocessor(&k.occ_part, k.partfn, (int)k.threads(), k.dyn_smem));
-    int sm_smem = 0, max_optin = 0;
-    CK(ctx, cudaDeviceGetAttribute(&sm_smem, cudaDevAttrMaxSharedMemoryPerMultiprocessor, ctx->cfg.device));
-    CK(ctx, cudaDeviceGetAttribute(&max_optin, cudaDevAttrMaxSharedMemoryPerBlockOptin, ctx->cfg.device));
-    k.part_smem = k.dyn_smem;
-    if (k.occ_part >= 1) {
-      int64_t per = (int64_t)(sm_smem / k.occ_part) / 128 * 128;  // footprint per CTA
-      for (; per >= 128; per -= 128) {
-        const int64_t dyn = per - 1024 - (int64_t)pa.sharedSizeBytes;
-        if (dyn < (int64_t)k.dyn_smem) break;
-        if (dyn + (int64_t)pa.sharedSizeBytes > max_optin) continue;
-        CK(ctx, cudaFuncSetAttribute(k.partfn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)dyn));
-        int occ = 0;
-        CK(ctx, cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k.partfn, (int)k.threads(), (size_t)dyn));
-        if (occ == k.occ_part) {
-          k.part_smem = (uint32_t)dyn;
-          break;
-        }
-      }
-      if (k.part_smem > 48 * 1024 || k.dyn_smem > 48 * 1024)
-        CK(ctx, cudaFuncSetAttribute(k.partfn, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                     (int)std::max(k.part_smem, k.dyn_smem)));
-    }
-  }
   accel_demand dem;
   int rc = accel_demand_of(&ctx->caps, k.threads(), (uint32_t)k.num_regs,
                            (uint32_t)(k.static_smem + k.dyn_smem), 1, 1, &dem);
@@ -1134,8 +1005,6 @@ int accel_kernel_info_get(accel_ctx* ctx, int32_t kernel_id, accel_kernel_info* 
   out->static_smem = k.static_smem;
   out->occ_persistent = k.occ_p;
   out->occ_native = k.occ_n;
-  out->occ_partition = k.occ_part;
-  out->partition_smem = k.part_smem;
   return ACCEL_OK;
 }
 
@@ -1320,18 +1189,6 @@ int accel_launch_times(accel_ctx* ctx, uint64_t request_id, float* ms_out, uint3
   if (!r->done) return ACCEL_ENOTREADY;
   if (r->ev_launch.empty()) return ctx->fail(ACCEL_EINVAL, "request had no ACCEL_REQ_LAUNCH_EVENTS");
   const uint32_t m = std::min<uint32_t>(n, r->n_desc);
-  if (r->part) {
-    // PARTITION: one grid per step, events around it; a launch gets the
-    // step's time divided by its launches
-    for (const Step& st : r->steps) {
-      const uint32_t end = st.first + st.repeat;
-      float ms = 0.f;
-      CK(ctx, cudaEventElapsedTime(&ms, r->ev_launch[st.first], r->ev_launch[end]));
-      for (uint32_t i = st.first; i < end && i < m; ++i) ms_out[i] = ms / (float)st.repeat;
-    }
-    *n_out = m;
-    return ACCEL_OK;
-  }
   for (uint32_t i = 0; i < m; ++i)
     CK(ctx, cudaEventElapsedTime(&ms_out[i], r->ev_launch[i], r->ev_launch[i + 1]));
   *n_out = m;

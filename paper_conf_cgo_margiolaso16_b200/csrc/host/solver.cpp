@@ -256,76 +256,3 @@ extern "C" int accel_solve(const accel_caps* caps, const accel_demand* d, int32_
   for (int i = 0; i < k; ++i) quota_out[i] = (uint32_t)n[i];
   return ACCEL_OK;
 }
-
-// SM-granular partitioning (DESIGN.md R-part-1..4; Fig. 3b, lines
-// 441-445: A's work-groups on CU0/1, B's on CU2/3).  The §3 rule with whole SMs
-// as the unit: s_i = floor(S w_i / W) capped at ceil(G_i / c_i), >= 1; class
-// decrement while the floors overshoot S; class-symmetric greedy +1 SM.  c_i =
-// CTAs of kernel i alone on one SM under the same model F.  Must agree
-// exactly with oracle/solver_ref.py solve_sms.
-extern "C" int accel_solve_sms(const accel_caps* caps, const accel_demand* d, int32_t k, uint32_t* sms_out,
-                               uint32_t* ctas_per_sm_out) {
-  if (k < 0 || (k > 0 && (!d || !sms_out))) return ACCEL_EINVAL;
-  const Caps c = caps_of(caps);
-  Caps one = c;
-  one.sms = 1;
-  std::vector<Req> rs(k);
-  std::vector<int64_t> per(k), cap(k), s(k, 0);
-  for (int i = 0; i < k; ++i) {
-    rs[i] = Req{d[i].thr, d[i].regs, d[i].smem, d[i].cta, d[i].grid_vgs, d[i].weight ? d[i].weight : 1};
-    if (!valid(rs[i], c)) return ACCEL_ENOFIT;
-    int64_t n = 0;
-    while (n < c.ctas && feasible(std::vector<Req>{rs[i]}, std::vector<int64_t>{n + 1}, one)) ++n;
-    per[i] = n;
-    cap[i] = cdiv(rs[i].g, n);
-  }
-  std::vector<std::vector<int>> cls;
-  for (int i = 0; i < k; ++i) {
-    bool placed = false;
-    for (auto& m : cls)
-      if (rs[m[0]].same(rs[i])) {
-        m.push_back(i);
-        placed = true;
-        break;
-      }
-    if (!placed) cls.push_back({i});
-  }
-  int64_t W = 0;
-  for (auto& r : rs)
-    if (r.g > 0) W += r.w;
-  for (int i = 0; i < k; ++i)
-    if (rs[i].g > 0) s[i] = std::max<int64_t>(1, std::min<int64_t>((c.sms * rs[i].w) / W, cap[i]));
-  auto total = [&]() {
-    int64_t t = 0;
-    for (int64_t v : s) t += v;
-    return t;
-  };
-  while (total() > c.sms) {
-    int best = -1;
-    for (size_t ci = 0; ci < cls.size(); ++ci) {
-      const int i = cls[ci][0];
-      if (s[i] <= 1) continue;
-      // s_i / w_i >= s_b / w_b : later class wins ties
-      if (best < 0 || s[i] * rs[cls[best][0]].w >= s[cls[best][0]] * rs[i].w) best = (int)ci;
-    }
-    if (best < 0) break;
-    for (int i : cls[best]) s[i] -= 1;
-  }
-  for (;;) {
-    bool accepted = false;
-    for (auto& m : cls) {
-      bool room = total() + (int64_t)m.size() <= c.sms;
-      for (int i : m)
-        if (s[i] + 1 > cap[i]) room = false;
-      if (!room) continue;
-      for (int i : m) s[i] += 1;
-      accepted = true;
-    }
-    if (!accepted) break;
-  }
-  for (int i = 0; i < k; ++i) {
-    sms_out[i] = (uint32_t)s[i];
-    if (ctas_per_sm_out) ctas_per_sm_out[i] = (uint32_t)per[i];
-  }
-  return ACCEL_OK;
-}

@@ -28,8 +28,6 @@ __global__ void desc_init_kernel(const InitParams p, uint32_t n_desc) {
   if (i == 0 && p.ctl != nullptr) {
     p.ctl->live = p.live_init;
     p.ctl->cur = 0;
-    p.ctl->sm_quota = p.sm_quota_init;
-    p.ctl->sm_count = 0;
     p.ctl->done_vgs = 0;
   }
   if (i >= n_desc) return;
@@ -49,11 +47,7 @@ __global__ void desc_init_kernel(const InitParams p, uint32_t n_desc) {
   d->ctl = p.ctl;
   d->coverage = p.coverage ? p.coverage + st.cov_offset + (size_t)r * st.total : nullptr;
   d->trace = p.trace ? p.trace + st.cov_offset + (size_t)r * st.total : nullptr;
-  d->governed = (s == p.main_step && p.owner == nullptr) ? 1u : 0u;
-  d->tok = p.tok;
-  d->owner = p.owner;
-  d->last_step = s + 1 == p.n_steps ? 1u : 0u;
-  d->ctas_per_sm = st.ctas_per_sm;
+  d->governed = s == p.main_step ? 1u : 0u;
   d->order = st.order;
   d->t_first = ULLONG_MAX;
   d->t_last = 0;
@@ -63,27 +57,20 @@ __global__ void desc_init_kernel(const InitParams p, uint32_t n_desc) {
   d->evicted = 0;
   d->draining = 0;
   d->last_live = 0;
-  d->topped = p.owner != nullptr ? 1u : 0u;   // PARTITION: any grid may serve any launch
+  d->topped = 0;
   d->req_idx = i;
   d->has_prev = i > 0 ? 1u : 0u;
   d->qa = st.qa0;
 }
 
 // Request completion: wait until the last launch completed if another grid
-// may still be serving it.  PARTITION: then hand back every SM the request
-// still owns (a safety net: its CTAs free their SMs when they finish).
-__global__ void join_kernel(const Desc* last, uint32_t nsm) {
+// (a RESOLVE top-up) may still be serving it.
+__global__ void join_kernel(const Desc* last) {
   if (threadIdx.x == 0 && ld_volatile(&last->topped)) wait_complete(last);
-  __syncwarp();
-  if (last->owner != nullptr)
-    for (uint32_t sm = threadIdx.x; sm < nsm; sm += 32) {
-      const uint32_t o = ld_volatile(&last->owner[sm]);
-      if ((o & ~(kOwnRel | kOwnClaim)) == last->tok) atomicCAS(&last->owner[sm], o, 0u);
-    }
 }
 
-cudaError_t launch_join(const Desc* last, uint32_t nsm, cudaStream_t s) {
-  join_kernel<<<1, 32, 0, s>>>(last, nsm);
+cudaError_t launch_join(const Desc* last, cudaStream_t s) {
+  join_kernel<<<1, 32, 0, s>>>(last);
   return cudaGetLastError();
 }
 
@@ -101,8 +88,7 @@ accel_kernel_desc make_desc(const char* name) {
   d.persistent_fn = reinterpret_cast<const void*>(&accel_persistent<T, false>);
   d.persistent_resolve_fn = reinterpret_cast<const void*>(&accel_persistent<T, true>);
   d.native_fn = reinterpret_cast<const void*>(&accel_native<T>);
-  d.topup_fn = reinterpret_cast<const void*>(&accel_topup<T, false>);
-  d.partition_fn = reinterpret_cast<const void*>(&accel_topup<T, true>);
+  d.topup_fn = reinterpret_cast<const void*>(&accel_topup<T>);
   d.block = accel_dim3{(uint32_t)T::kThreads, 1u, 1u};
   d.dyn_smem = T::kDynSmem;
   d.regs = 0;
@@ -119,7 +105,9 @@ struct Builtin {
 const Builtin kBuiltins[] = {
     {"mop", &make_desc<Mop>},
     {"stencil", &make_desc<Stencil>},
+    {"stencil_x", &make_desc<StencilX>},
     {"histo", &make_desc<Histo>},
+    {"histo_wide", &make_desc<HistoWide>},
     {"bfs", &make_desc<Bfs>},
     {"cutcp", &make_desc<Cutcp>},
     {"tpacf", &make_desc<Tpacf>},

@@ -7,22 +7,34 @@
 // completes launch r (done[r] counter, threadfence reduction) runs the "final"
 // step: sat[b] = min(hist, 255), and zeroes the other half of hist for the
 // next launch.  No cross-CTA waiting: the last finisher does the tail work.
+//
+// Two instantiations (up to 16,384 bins at the B200 default):
+//   histo       u32 private counters, <= 4,096 bins, 16 KB smem
+//   histo_wide  16-bit private counters packed two per word (bin b in the
+//               half b & 1 of word b >> 1: a shared-memory add of 1 << 16
+//               never carries into the other half while a VG counts fewer
+//               than 65,536 samples), <= 16,384 bins in 32 KB smem, u32
+//               samples only.
 #pragma once
 #include "../device/dispatch.cuh"
 #include "accel_tenants.h"
 
 namespace accel {
 
-struct Histo {
+template <bool kPacked>
+struct HistoT {
   using Args = accel_histo_args;
   static constexpr int kThreads = 256;
   static constexpr uint32_t kChunk = 1;
   static constexpr int kMinBlocks = 6;    // <= 40 regs in both modes
-  static constexpr uint32_t kMaxBins = 4096;
-  static constexpr uint32_t kDynSmem = kMaxBins * sizeof(uint32_t);  // 16 KB
+  static constexpr uint32_t kMaxBins = kPacked ? 16384 : 4096;
+  static constexpr uint32_t kWords = kPacked ? kMaxBins / 2 : kMaxBins;
+  static constexpr uint32_t kDynSmem = kWords * sizeof(uint32_t);  // 16 / 32 KB
 
   static __device__ __forceinline__ void count4(uint32_t* h, uint32_t w, uint32_t sb) {
-    if (sb == 1) {
+    if constexpr (kPacked) {
+      atomicAdd(&h[w >> 1], 1u << ((w & 1u) << 4));
+    } else if (sb == 1) {
 #pragma unroll
       for (int k = 0; k < 4; ++k) atomicAdd(&h[(w >> (8 * k)) & 0xffu], 1u);
     } else {
@@ -34,8 +46,9 @@ struct Histo {
     uint32_t* h = reinterpret_cast<uint32_t*>(smem);
     __shared__ bool s_last;
     const uint32_t bins = a.bins;
+    const uint32_t words = kPacked ? (bins + 1u) >> 1 : bins;
     const uint32_t r = vb.launch_idx;
-    for (uint32_t b = threadIdx.x; b < bins; b += kThreads) h[b] = 0u;
+    for (uint32_t b = threadIdx.x; b < words; b += kThreads) h[b] = 0u;
     __syncthreads();
 
     const uint32_t sb = a.sample_bytes;
@@ -71,13 +84,21 @@ struct Histo {
     for (uint64_t i = lo + nvec * per_vec + threadIdx.x; i < hi; i += kThreads) {
       const uint32_t s = sb == 1 ? (uint32_t)reinterpret_cast<const uint8_t*>(base)[i]
                                  : reinterpret_cast<const uint32_t*>(base)[i];
-      atomicAdd(&h[s], 1u);
+      if constexpr (kPacked)
+        atomicAdd(&h[s >> 1], 1u << ((s & 1u) << 4));
+      else
+        atomicAdd(&h[s], 1u);
     }
     __syncthreads();
     uint32_t* gh = a.hist + (r & 1u) * bins;
-    for (uint32_t b = threadIdx.x; b < bins; b += kThreads) {
+    for (uint32_t b = threadIdx.x; b < words; b += kThreads) {
       const uint32_t c = h[b];
-      if (c) atomicAdd(&gh[b], c);
+      if constexpr (kPacked) {
+        if (c & 0xffffu) atomicAdd(&gh[2 * b], c & 0xffffu);
+        if (c >> 16) atomicAdd(&gh[2 * b + 1], c >> 16);   // bin 2b+1 < bins whenever counted
+      } else {
+        if (c) atomicAdd(&gh[b], c);
+      }
     }
     // final step by the VG that completes launch r
     __threadfence();
@@ -98,5 +119,8 @@ struct Histo {
     }
   }
 };
+
+using Histo = HistoT<false>;
+using HistoWide = HistoT<true>;
 
 }  // namespace accel

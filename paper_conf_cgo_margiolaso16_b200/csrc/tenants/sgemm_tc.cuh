@@ -81,6 +81,19 @@ struct SgemmSplit {
     float* __restrict__ lo = s1 ? a.lo1 : a.lo0;
     const uint64_t n = s1 ? a.n1 : a.n0;
     const uint64_t base = (uint64_t)(s1 ? vb.linear - g0 : vb.linear) * kPerVG;
+    if (a.cols != a.ld) {   // K % 4 != 0: rows of the outputs padded to ld
+#pragma unroll
+      for (int u = 0; u < 16; ++u) {
+        const uint64_t i = base + (uint64_t)(u * kThreads + threadIdx.x);
+        if (i < n) {
+          const uint64_t o = (i / a.cols) * a.ld + i % a.cols;
+          const float v = __ldcs(src + i), h = hi_of(v);
+          hi[o] = h;
+          lo[o] = v - h;
+        }
+      }
+      return;
+    }
 #pragma unroll
     for (int u = 0; u < 4; ++u) {
       const uint64_t i = base + (uint64_t)(u * kThreads + threadIdx.x) * 4;

@@ -26,12 +26,18 @@
 
 namespace accel {
 
-struct Stencil {
+// kAligned: nx % 4 == 0 (kernel "stencil": every row starts 16-B aligned).
+// !kAligned: any nx (kernel "stencil_x"): the same tile staged with 4-B
+// cp.async copies, each column checked against nx, outputs stored per
+// element.  Two kernels rather than a branch: the ragged path's registers
+// would otherwise count against the aligned one (it spilled).
+template <bool kAligned>
+struct StencilT {
   using Args = accel_stencil_args;
   static constexpr int kThreads = 256;
   static constexpr int kTX = 128, kTY = 8, kTZ = 8;
   static constexpr uint32_t kChunk = 1;
-  static constexpr int kMinBlocks = 5;
+  static constexpr int kMinBlocks = kAligned ? 5 : 4;   // the ragged path needs a few more registers
   static constexpr int kRows = kTY + 2;                 // y halo
   static constexpr int kCols = kTX + 8;                 // x0-4 .. x0+131 (16-B multiples)
   static constexpr uint32_t kPlaneBytes = kRows * kCols * 4;          // 5440
@@ -102,10 +108,26 @@ struct Stencil {
     const long long off0 = (long long)(z0 - 1) * pstr + (long long)ys0 * nx + c0x;
     const long long off1 = (long long)(z0 - 1) * pstr + (long long)ys1 * nx + c1x;
     const uint32_t soff0 = 16u * (uint32_t)e0, soff1 = 16u * (uint32_t)e1;
+    // ragged x (nx % 4 != 0): a piece is four 4-B copies, column c + j read
+    // only when c + j < nx (c >= 0 is all-or-nothing: x0 - 4 is a multiple of 4)
+    auto piece4 = [&](uint32_t dst, long long off, int cx, bool okyz) {
+#pragma unroll
+      for (int j = 0; j < 4; ++j) {
+        const bool ok = okyz && cx >= 0 && cx + j < nx;
+        const float* src = ok ? in + (off + j) : in;
+        asm volatile("cp.async.ca.shared.global [%0], [%1], 4, %2;" ::"r"(dst + 4u * j), "l"(src), "r"(ok ? 4 : 0)
+                     : "memory");
+      }
+    };
     auto issue = [&](int p) {
       const uint32_t dst = sbase + (uint32_t)(p % kR) * kSlot;
       const int zs = z0 - 1 + p;
       const bool zok = zs >= 0 && zs < nz;          // uniform
+      if constexpr (!kAligned) {
+        piece4(dst + soff0, off0 + (long long)p * pstr, c0x, zok && ys0 >= 0 && ys0 < ny);
+        if (has1) piece4(dst + soff1, off1 + (long long)p * pstr, c1x, zok && ys1 >= 0 && ys1 < ny);
+        return;
+      }
       const bool ok0 = okxy0 && zok;
       const float* s0 = ok0 ? in + (off0 + (long long)p * pstr) : in;
       asm volatile("cp.async.cg.shared.global [%0], [%1], 16, %2;" ::"r"(dst + soff0), "l"(s0), "r"(ok0 ? 16 : 0)
@@ -212,7 +234,15 @@ struct Stencil {
           arrive_full(pz + kD + 1);
         }
       }
-      if (active) *reinterpret_cast<float4*>(po) = o;
+      if constexpr (kAligned) {
+        if (active) *reinterpret_cast<float4*>(po) = o;
+      } else if (active) {
+        const int xr0 = nx - (x0 + 4 * lane);   // >= 1 elements of this vector in range
+        po[0] = o.x;
+        if (xr0 > 1) po[1] = o.y;
+        if (xr0 > 2) po[2] = o.z;
+        if (xr0 > 3) po[3] = o.w;
+      }
       po += pstr;
       zm = cur;
       cur = zp;
@@ -222,5 +252,8 @@ struct Stencil {
   }
 
 };
+
+using Stencil = StencilT<true>;
+using StencilX = StencilT<false>;
 
 }  // namespace accel

@@ -37,12 +37,25 @@ def _cdiv(a: int, b: int) -> int:
     return -(-a // b)
 
 
+def _measured_peaks() -> dict:
+    """MEASURED_PEAKS.json (driver-written, repo root); B200_PROFILING.md's
+    fallback figures when it is absent."""
+    import json
+    import os
+    p = os.path.join(os.path.dirname(os.path.dirname(os.path.abspath(__file__))), "MEASURED_PEAKS.json")
+    try:
+        with open(p) as f:
+            return json.load(f)
+    except OSError:
+        return {"hbm_gbs": 6650.0, "bf16_tflops": 1590.0, "sm_max_mhz": 1965.0}
+
+
 # Roofline peaks for the non-HBM tenants (DESIGN.md §6): FP32 SIMT derived from
-# the guide's unit counts (148 SM x 128 FP32 lanes x 2 flop x 1.965 GHz); TF32
-# tensor = the measured bf16 dense peak (MEASURED_PEAKS.json, 1678.1 TF/s
-# burst) x the nominal TF32/BF16 ratio 1/2.
-FP32_SIMT_TFLOPS = 148 * 128 * 2 * 1.965e9 / 1e12
-TF32_TENSOR_TFLOPS = 1678.1 / 2
+# the guide's unit counts (148 SM x 128 FP32 lanes x 2 flop x max SM clock);
+# TF32 tensor = the measured dense bf16 peak x the nominal TF32/BF16 ratio 1/2.
+PEAKS = _measured_peaks()
+FP32_SIMT_TFLOPS = 148 * 128 * 2 * PEAKS.get("sm_max_mhz", 1965.0) * 1e6 / 1e12
+TF32_TENSOR_TFLOPS = PEAKS["bf16_tflops"] / 2
 
 
 @dataclass
@@ -169,8 +182,6 @@ class StencilJob(Job):
     def __init__(self, d: dict, device="cuda"):
         super().__init__(name="stencil", device=torch.device(device))
         self.nx, self.ny, self.nz, self.sweeps = d["nx"], d["ny"], d["nz"], d["sweeps"]
-        if self.nx % 4:
-            raise ValueError("stencil needs nx % 4 == 0 (16-B rows)")
         n = self.nx * self.ny * self.nz
         self.inputs = {"a0": _dev(d["a0"].ravel(), self.device)}
         self.buf = [torch.empty(n, dtype=torch.float32, device=self.device) for _ in range(2)]
@@ -178,7 +189,8 @@ class StencilJob(Job):
         self.args = abi.accel_stencil_args(self.inputs["a0"].data_ptr(), self.buf[0].data_ptr(),
                                            self.buf[1].data_ptr(), self.nx, self.ny, self.nz, d["c0"], d["c1"])
         grid = (_cdiv(self.nx, self.TX), _cdiv(self.ny, self.TY), _cdiv(self.nz, self.TZ))
-        self.steps = [Step("stencil", grid, self.args, self.sweeps)]
+        # rows 16-B aligned (nx % 4 == 0): cp.async 16-B pieces; else the any-nx kernel
+        self.steps = [Step("stencil" if self.nx % 4 == 0 else "stencil_x", grid, self.args, self.sweeps)]
 
     def result(self):
         return {"a": _np(self.out["a"], np.float32).reshape(self.nz, self.ny, self.nx)}
@@ -193,8 +205,12 @@ class HistoJob(Job):
     def __init__(self, d: dict, device="cuda"):
         super().__init__(name="histo", device=torch.device(device))
         self.n, self.bins, self.iters, self.sb = d["n"], d["bins"], d["iters"], d["sample_bytes"]
-        assert self.bins <= 4096 and (self.sb == 4 or self.bins == 256)
-        self.per_vg = 4096 if self.sb == 1 else 16384
+        if not (1 <= self.bins <= 16384 and (self.sb == 4 or self.bins == 256)):
+            raise ValueError("histo: 1..16384 bins; u8 samples need 256 bins")
+        # > 4096 bins: the packed 16-bit private histogram (VGs < 65536 samples)
+        self.kernel = "histo" if self.bins <= 4096 else "histo_wide"
+        self.per_vg = 4096 if self.sb == 1 else d.get("per_vg", 16384)
+        assert self.per_vg % 4096 == 0 and (self.kernel == "histo" or self.per_vg < 65536)
         self.inputs = {"samples": _dev(d["samples"], self.device)}
         self.hist = torch.zeros(2 * self.bins, dtype=torch.int32, device=self.device)
         self.sat = torch.zeros(self.bins, dtype=torch.uint8, device=self.device)
@@ -205,7 +221,7 @@ class HistoJob(Job):
                                          self.per_vg, self.hist.data_ptr(), self.sat.data_ptr(),
                                          self.done.data_ptr())
         self.clears = [(self.hist, 0), (self.done, 0)]
-        self.steps = [Step("histo", (_cdiv(self.n, self.per_vg), 1, 1), self.args, self.iters)]
+        self.steps = [Step(self.kernel, (_cdiv(self.n, self.per_vg), 1, 1), self.args, self.iters)]
 
     def result(self):
         return {"counts": _np(self.out["counts"], np.uint32), "sat": _np(self.sat, np.uint8)}
@@ -413,17 +429,16 @@ class SgemmTcJob(Job):
     def __init__(self, d: dict, device="cuda"):
         super().__init__(name="sgemm", device=torch.device(device))
         self.m, self.n, self.k = d["m"], d["n"], d["k"]
-        if self.k % 4:
-            raise ValueError("sgemm needs k % 4 == 0 (16-B rows)")
         self.inputs = {"a": _dev(d["a"].ravel(), self.device), "b": _dev(d["b"].ravel(), self.device)}
         m, n, k = self.m, self.n, self.k
+        kp = _cdiv(k, 4) * 4   # hi/lo row stride: 16-B aligned rows for TMA
         self.split = {x: torch.empty(sz, dtype=torch.float32, device=self.device)
-                      for x, sz in (("a_hi", m * k), ("a_lo", m * k), ("b_hi", n * k), ("b_lo", n * k))}
+                      for x, sz in (("a_hi", m * kp), ("a_lo", m * kp), ("b_hi", n * kp), ("b_lo", n * kp))}
         maps = b"".join([
-            abi.accel_tma_map_2d(self.split["a_hi"].data_ptr(), k, m, 4 * k, 32, 128),
-            abi.accel_tma_map_2d(self.split["a_lo"].data_ptr(), k, m, 4 * k, 32, 128),
-            abi.accel_tma_map_2d(self.split["b_hi"].data_ptr(), k, n, 4 * k, 32, 256),
-            abi.accel_tma_map_2d(self.split["b_lo"].data_ptr(), k, n, 4 * k, 32, 256)])
+            abi.accel_tma_map_2d(self.split["a_hi"].data_ptr(), k, m, 4 * kp, 32, 128),
+            abi.accel_tma_map_2d(self.split["a_lo"].data_ptr(), k, m, 4 * kp, 32, 128),
+            abi.accel_tma_map_2d(self.split["b_hi"].data_ptr(), k, n, 4 * kp, 32, 256),
+            abi.accel_tma_map_2d(self.split["b_lo"].data_ptr(), k, n, 4 * kp, 32, 256)])
         self.tmaps = torch.frombuffer(bytearray(maps), dtype=torch.uint8).to(self.device)
         self.c = torch.empty(m * n, dtype=torch.float32, device=self.device)
         self.out = {"c": self.c}
@@ -432,7 +447,7 @@ class SgemmTcJob(Job):
         self.args_s = abi.accel_sgemm_split_args(self.inputs["a"].data_ptr(), s["a_hi"].data_ptr(),
                                                  s["a_lo"].data_ptr(), m * k,
                                                  self.inputs["b"].data_ptr(), s["b_hi"].data_ptr(),
-                                                 s["b_lo"].data_ptr(), n * k)
+                                                 s["b_lo"].data_ptr(), n * k, k, kp)
         self.args_tc = abi.accel_sgemm_tc_args(self.tmaps.data_ptr(), self.c.data_ptr(), m, n, k)
         self.main_step = 1
         self.steps = [Step("sgemm_split", (_cdiv(m * k, 4096) + _cdiv(n * k, 4096), 1, 1), self.args_s, 1),
@@ -444,7 +459,7 @@ class SgemmTcJob(Job):
     def work(self):
         f = 2.0 * self.m * self.n * self.k
         # roofline of the dominant (tc) launch: 3 tf32 products per algorithmic MAC
-        return {"flops": f, "flops_per_launch": f, "bound": "tensor", "launches": 3, "skip_launches": 2,
+        return {"flops": f, "flops_per_launch": f, "bound": "tensor", "launches": 2, "skip_launches": 1,
                 "mma_flops": 3 * f, "peak_tflops": TF32_TENSOR_TFLOPS}
 
 

@@ -26,7 +26,7 @@ def main():
     ap.add_argument("--size", default="default")
     ap.add_argument("--reps", type=int, default=5)
     ap.add_argument("--chunk", type=int, default=0, help="override VGs per dequeue for all kernels")
-    ap.add_argument("--policy", default="both", choices=["static", "resolve", "partition", "both", "all"])
+    ap.add_argument("--policy", default="both", choices=["static", "resolve", "both"])
     args = ap.parse_args()
     from paper_conf_cgo_margiolaso16_b200 import abi as _abi
     chunks = {n: args.chunk for n in _abi.accel_builtin_names()} if args.chunk else None
@@ -37,11 +37,9 @@ def main():
         d = synth.preset(t, args.size, seed=1)
         job = make_job(t, d)
         res = {}
-        pols = {"static": [abi.POLICY_STATIC], "resolve": [abi.POLICY_RESOLVE], "partition": [abi.POLICY_PARTITION],
-                "both": [abi.POLICY_STATIC, abi.POLICY_RESOLVE],
-                "all": [abi.POLICY_STATIC, abi.POLICY_RESOLVE, abi.POLICY_PARTITION]}[args.policy]
-        pname = {abi.POLICY_STATIC: "persistent", abi.POLICY_RESOLVE: "persistent_resolve",
-                 abi.POLICY_PARTITION: "persistent_partition"}
+        pols = {"static": [abi.POLICY_STATIC], "resolve": [abi.POLICY_RESOLVE],
+                "both": [abi.POLICY_STATIC, abi.POLICY_RESOLVE]}[args.policy]
+        pname = {abi.POLICY_STATIC: "persistent", abi.POLICY_RESOLVE: "persistent_resolve"}
         runs = [(abi.MODE_NATIVE, "native", abi.POLICY_STATIC)] + [(abi.MODE_SHARED, pname[p], p) for p in pols]
         for mode, name, pol in runs:
             acc.set_mode(mode, pol)
@@ -68,7 +66,7 @@ def main():
                 f = w.get("flops_per_launch", w.get("flops"))
                 r["TFLOPs_mean"] = f / r["launch_ms_mean"] / 1e9
             res[name] = r
-        for nm in ("persistent", "persistent_resolve", "persistent_partition"):
+        for nm in ("persistent", "persistent_resolve"):
             if nm in res:
                 res["overhead" + nm[len("persistent"):]] = res[nm]["elapsed_ms"] / res["native"]["elapsed_ms"] - 1
         if "persistent_resolve" in res:

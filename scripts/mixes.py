@@ -42,9 +42,8 @@ from paper_conf_cgo_margiolaso16_b200.runtime import Accel  # noqa: E402
 
 TENANTS = ["bfs", "cutcp", "stencil", "tpacf", "histo", "spmv", "sgemm", "mriq"]
 MODES = [("native", abi.MODE_NATIVE, abi.POLICY_STATIC), ("resolve", abi.MODE_SHARED, abi.POLICY_RESOLVE),
-         ("static", abi.MODE_SHARED, abi.POLICY_STATIC), ("partition", abi.MODE_SHARED, abi.POLICY_PARTITION),
-         ("fair", abi.MODE_SHARED, abi.POLICY_FAIR)]
-SHARED = ["resolve", "static", "partition", "fair"]
+         ("static", abi.MODE_SHARED, abi.POLICY_STATIC), ("fair", abi.MODE_SHARED, abi.POLICY_FAIR)]
+SHARED = ["resolve", "static", "fair"]
 
 
 def gm(xs):

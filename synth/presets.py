@@ -21,14 +21,14 @@ PRESETS: dict[str, dict[str, dict]] = {
         "default": dict(n=1 << 26, block=256),
     },
     "stencil": {
-        "tiny": dict(nx=72, ny=21, nz=19, sweeps=3),
+        "tiny": dict(nx=70, ny=21, nz=19, sweeps=3),
         "small": dict(nx=64, ny=64, nz=64, sweeps=100),
         "default": dict(nx=512, ny=512, nz=64, sweeps=100),
     },
     "histo": {
         "tiny": dict(n=100_003, bins=256, iters=2, sample_bytes=1),
         "small": dict(n=1 << 18, bins=256, iters=20, sample_bytes=1),
-        "default": dict(n=1 << 25, bins=4096, iters=20, sample_bytes=4),
+        "default": dict(n=1 << 24, bins=16384, iters=100, sample_bytes=4),
     },
     "bfs": {
         "tiny": dict(nv=3000),

@@ -10,7 +10,10 @@ pytestmark = pytest.mark.gpu
 
 
 @pytest.mark.parametrize("size,over", [("tiny", dict(m=256, n=512, k=64)), ("tiny", {}),
-                                       ("small", {}), ("tiny", dict(m=129, n=257, k=36))])
+                                       ("small", {}), ("tiny", dict(m=129, n=257, k=36)),
+                                       ("tiny", dict(m=130, n=140, k=70)),     # k % 4 == 2: padded hi/lo rows
+                                       ("tiny", dict(m=64, n=33, k=33)),       # k % 4 == 1, k not a slab multiple
+                                       ("tiny", dict(m=5, n=7, k=3))])
 def test_sgemm_tc(acc_tiny_caps, oracle_lib, size, over):
     from paper_conf_cgo_margiolaso16_b200.jobs import SgemmTcJob
     d = synth.preset("sgemm", size, **over)

@@ -82,6 +82,9 @@ def test_mop_small_fullcaps(acc, oracle_lib):
 
 # ---------------------------------------------------------------- stencil
 @pytest.mark.parametrize("size,over", [("tiny", {}), ("tiny", dict(nx=132, ny=9, nz=17, sweeps=2)),
+                                       ("tiny", dict(nx=67, ny=13, nz=10, sweeps=3)),   # nx % 4 == 3
+                                       ("tiny", dict(nx=129, ny=8, nz=9, sweeps=2)),    # one column past a tile
+                                       ("tiny", dict(nx=2, ny=5, nz=4, sweeps=2)),      # all faces
                                        ("small", dict(sweeps=10))])
 def test_stencil(acc_tiny_caps, oracle_lib, size, over):
     from paper_conf_cgo_margiolaso16_b200.jobs import StencilJob
@@ -110,6 +113,8 @@ def test_stencil_default_sampled(acc, oracle_lib):
 
 # ---------------------------------------------------------------- histo
 @pytest.mark.parametrize("size,over", [("tiny", {}), ("tiny", dict(bins=4096, sample_bytes=4)),
+                                       ("tiny", dict(bins=16384, sample_bytes=4)),      # histo_wide
+                                       ("tiny", dict(bins=10007, sample_bytes=4, iters=3)),  # odd bin count
                                        ("small", {}), ("small", dict(n=(1 << 18) + 13, iters=3))])
 def test_histo(acc_tiny_caps, oracle_lib, size, over):
     from paper_conf_cgo_margiolaso16_b200.jobs import HistoJob
@@ -122,12 +127,27 @@ def test_histo(acc_tiny_caps, oracle_lib, size, over):
 
 
 def test_histo_default(acc, oracle_lib):
+    """SURVEY §8(d).1 B200 default: 2^24 u32 samples, 16,384 bins (histo_wide)."""
     from paper_conf_cgo_margiolaso16_b200.jobs import HistoJob
     d = synth.preset("histo", "default", iters=3)
+    assert d["n"] == 1 << 24 and d["bins"] == 16384
     nat, sh, _ = run_modes(acc, lambda: HistoJob(d))
     counts, sat = oracle_lib.histo(d)
     assert np.array_equal(sh["counts"], counts) and np.array_equal(nat["counts"], counts)
-    assert np.array_equal(sh["sat"], sat)
+    assert np.array_equal(sh["sat"], sat) and np.array_equal(nat["sat"], sat)
+    assert int(counts.sum()) == d["n"]
+
+
+@pytest.mark.parametrize("per_vg", [8192, 32768, 61440])
+def test_histo_wide_vg_sizes(acc_tiny_caps, oracle_lib, per_vg):
+    """16-bit packed counters stay exact up to the largest allowed VG (the
+    bins near the Gaussian peak take thousands of counts per VG)."""
+    from paper_conf_cgo_margiolaso16_b200.jobs import HistoJob
+    d = dict(synth.preset("histo", "small", bins=16384, sample_bytes=4, n=(1 << 19) + 77, iters=2), per_vg=per_vg)
+    nat, sh, _ = run_modes(acc_tiny_caps, lambda: HistoJob(d))
+    counts, sat = oracle_lib.histo(d)
+    for r in (nat, sh):
+        assert np.array_equal(r["counts"], counts) and np.array_equal(r["sat"], sat)
 
 
 # ---------------------------------------------------------------- mixes

@@ -177,105 +177,6 @@ def test_step_quota():
     assert S.step_quota([main, other], 0, big_smem) == 148  # one 191-KB CTA per SM
 
 
-# ---- SM-granular partition (DESIGN.md R-part-1..4) -------------------------
-
-def test_partition_fig3_worked_example():
-    """Fig. 3b (lines 441-445) IS an SM partition: 4 CUs, each fits one WG of A
-    (12 WGs) or B (8 WGs); A gets CU0/CU1 and B CU2/CU3 -> 2 SMs each."""
-    caps = S.Caps(sms=4, thr_per_sm=256)
-    a = S.demand_of(256, 32, 0, 12, caps=caps)
-    b = S.demand_of(256, 32, 0, 8, caps=caps)
-    assert S.solve_sms([a, b], caps) == ([2, 2], [1, 1])
-    # alone, A takes every CU (standard FCFS reservation, lines 397-398)
-    assert S.solve_sms([a], caps) == ([4], [1])
-
-
-@pytest.mark.parametrize("block,regs,smem", [
-    (256, 32, 0), (256, 64, 0), (128, 255, 0), (256, 32, 100000), (96, 40, 0),
-    (1024, 32, 0), (128, 72, 16384), (64, 16, 48000), (512, 128, 0), (32, 255, 8000),
-])
-def test_partition_ctas_per_sm_is_occupancy(occ, block, regs, smem):
-    """c_i equals NVIDIA's occupancy calculator (a library pin), and K = 1
-    gives every SM up to ceil(G / c)."""
-    per_sm = occ(block, regs, 0, smem)
-    d = S.demand_of(block, regs, smem, 10 ** 6)
-    assert S.ctas_per_sm(d) == per_sm
-    for g in (1, per_sm, per_sm + 1, 148 * per_sm - 1, 10 ** 6):
-        dg = S.demand_of(block, regs, smem, g)
-        assert S.solve_sms([dg]) == ([min(148, -(-g // per_sm))], [per_sm])
-
-
-def test_partition_closed_forms():
-    d = S.demand_of(256, 32, 0, 10 ** 6)
-    # equal split of 148 SMs: 148 = 4 * 37, 3 * 49 + 1 (the odd SM stays free:
-    # identical requests get identical shares), 8 * 18 + 4
-    assert S.solve_sms([d] * 4)[0] == [37] * 4
-    assert S.solve_sms([d] * 3)[0] == [49] * 3
-    assert S.solve_sms([d] * 8)[0] == [18] * 8
-    # distinct requests take the leftovers in arrival order
-    ds = [S.demand_of(256, 32 + 8 * i, 0, 10 ** 6) for i in range(3)]
-    assert S.solve_sms(ds)[0] == [50, 49, 49]
-    # a small grid caps the share; the others take the surplus
-    small = S.demand_of(256, 32, 0, 16)  # c = 8 -> 2 SMs suffice
-    big = S.demand_of(128, 40, 0, 10 ** 6)
-    assert S.solve_sms([small, big])[0] == [2, 146]
-    # weights scale the share (lines 388-393)
-    a = S.demand_of(256, 32, 0, 10 ** 6, weight=3)
-    b = S.demand_of(256, 32, 0, 10 ** 6, weight=1)
-    assert S.solve_sms([a, b])[0] == [111, 37]
-
-
-def _partition_invariants(ds, s, c, caps):
-    assert sum(s) <= caps.sms or all(x <= 1 for x in s)
-    for d, x, ci in zip(ds, s, c):
-        assert ci == S.ctas_per_sm(d, caps)
-        if d.grid_vgs == 0:
-            assert x == 0
-        else:
-            assert 1 <= x <= -(-d.grid_vgs // ci)
-    # identical requests get identical SM counts
-    for members in S.classes(ds):
-        assert len({s[i] for i in members}) == 1
-    # class-maximal: no class can take one more SM per member
-    for members in S.classes(ds):
-        if all(s[i] + 1 <= -(-ds[i].grid_vgs // c[i]) for i in members):
-            assert sum(s) + len(members) > caps.sms
-
-
-def test_partition_random_invariants_and_bruteforce():
-    r = random.Random(21)
-    for trial in range(400):
-        caps = S.Caps(sms=r.randint(1, 12), thr_per_sm=r.choice([512, 1024, 2048]))
-        k = r.randint(1, 4)
-        ds = []
-        while len(ds) < k:
-            try:
-                ds.append(S.demand_of(r.choice([64, 128, 256]), r.choice([32, 64]), r.choice([0, 4096]),
-                                      r.randint(0, 60), r.choice([1, 1, 2]), caps=caps))
-            except S.NoFit:
-                pass
-        if r.random() < 0.3:
-            ds.append(ds[0])
-        s, c = S.solve_sms(ds, caps)
-        _partition_invariants(ds, s, c, caps)
-        if sum(1 for d in ds if d.grid_vgs > 0) > caps.sms:
-            continue
-        # brute force: the best achievable min over requests of s_i / w_i
-        # (with every request >= 1 SM) is never above the solver's
-        caps_g = [max(1, -(-d.grid_vgs // ci)) if d.grid_vgs else 0 for d, ci in zip(ds, c)]
-        best = None
-        for cand in itertools.product(*[range(1 if g else 0, g + 1) for g in caps_g]):
-            if sum(cand) > caps.sms:
-                continue
-            v = min((x / d.weight for x, d in zip(cand, ds) if d.grid_vgs), default=0)
-            best = v if best is None else max(best, v)
-        got = min((x / d.weight for x, d in zip(s, ds) if d.grid_vgs), default=0)
-        assert got <= best + 1e-12
-        # unit weights, no duplicate class: the greedy is max-min optimal
-        if len(S.classes(ds)) == len(ds) and all(d.weight == 1 for d in ds):
-            assert got == pytest.approx(best)
-
-
 def test_placement_big_cta_not_starved():
     """R-solver-3 / R-place-1: small CTAs arriving first must not fragment
     every SM.  A GEMM whose CTA needs a whole SM (640 threads x 96 registers)

@@ -99,27 +99,6 @@ def test_metrics_equal():
         assert abi.accel_overlap(st, en) == pytest.approx(M.overlap(list(zip(st, en))), abs=1e-12)
 
 
-def test_partition_parity():
-    r = random.Random(5)
-    n = 0
-    for _ in range(3000):
-        caps = S.Caps(sms=r.choice([1, 2, 3, 5, 9, 148]), thr_per_sm=r.choice([512, 1024, 2048]),
-                      regs_per_sm=r.choice([32768, 65536]), smem_per_sm=r.choice([65536, 233472]),
-                      ctas_per_sm=r.choice([4, 8, 16, 32]))
-        try:
-            ds = _random_instance(r, caps, 8, 5000)
-        except S.NoFit:
-            continue
-        ref = S.solve_sms(ds, caps)
-        got = abi.accel_solve_sms([_to_c(d) for d in ds], _caps(caps))
-        assert (list(got[0]), list(got[1])) == (list(ref[0]), list(ref[1])), (caps, ds)
-        n += 1
-    assert n > 2500
-    caps = S.Caps(sms=4, thr_per_sm=256)
-    a, b = S.demand_of(256, 32, 0, 12, caps=caps), S.demand_of(256, 32, 0, 8, caps=caps)
-    assert abi.accel_solve_sms([_to_c(a), _to_c(b)], _caps(caps)) == ([2, 2], [1, 1])
-
-
 def test_fair_weights_closed_forms():
     """FAIR weights (DESIGN.md R-fair-2): 16 * (s_i / geomean s)^2, clamped to
     [1, 1024]; equal slowdowns -> equal (neutral) weights; unknown (<= 0) ->
