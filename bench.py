@@ -383,6 +383,11 @@ def run_rank(args, rank, world, local, ranks: Ranks) -> dict:
     dev = torch.device("cuda", local)
     jobs = [make_job(t, inputs[t], dev) for t in tenants]
     acc = Accel(device=local, mode=abi.MODE_SHARED)
+    # bfs: launch levels until the frontier is empty (depth + 1 launches,
+    # learned by one untimed probe run)
+    for j in jobs:
+        if hasattr(j, "fit_levels"):
+            j.fit_levels(acc)
     flush_buf = torch.empty(256 * 1024 * 1024 // 4, dtype=torch.float32, device=dev)  # > L2 (126 MB)
 
     def flush():

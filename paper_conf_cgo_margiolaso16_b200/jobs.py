@@ -258,6 +258,29 @@ class BfsJob(Job):
     def frontier_sizes(self):
         return _np(self.count, np.uint32)
 
+    def set_levels(self, levels: int) -> None:
+        """Re-size the request to `levels` level launches (same buffers)."""
+        self.levels = int(levels)
+        self.count = torch.zeros(self.levels + 1, dtype=torch.int32, device=self.device)
+        self.args.count = self.count.data_ptr()
+        self.clears = [(self.level, 0xFF), (self.count, 0)]
+        self.steps = [Step("bfs", (_cdiv(self.nv, 256), 1, 1), self.args, self.levels)]
+
+    def fit_levels(self, acc) -> int:
+        """Parboil's bfs launches levels until the frontier is empty.  Here the
+        whole launch sequence is one request (no host round trip per level),
+        so its length is the graph's depth + 1, learned once by a probe run of
+        this request through `acc` (untimed set-up, like knowing a stencil's
+        sweep count): launch l writes the size of frontier l + 1 to count[l+1];
+        the first empty one ends the search.  Returns the fitted launch count."""
+        acc.run([self])
+        c = self.frontier_sizes()
+        empty = [l for l in range(1, len(c)) if c[l] == 0]
+        if not empty:
+            raise RuntimeError(f"bfs deeper than {self.levels} levels")
+        self.set_levels(empty[0])
+        return self.levels
+
     def work(self):
         b = 16 * self.nv + 8 * self.ne
         return {"bytes": b, "bytes_per_launch": b / self.levels, "bound": "hbm", "launches": self.levels}

@@ -36,6 +36,8 @@ def main():
     for t in args.tenants:
         d = synth.preset(t, args.size, seed=1)
         job = make_job(t, d)
+        if hasattr(job, "fit_levels"):
+            job.fit_levels(acc)
         res = {}
         pols = {"static": [abi.POLICY_STATIC], "resolve": [abi.POLICY_RESOLVE],
                 "both": [abi.POLICY_STATIC, abi.POLICY_RESOLVE]}[args.policy]

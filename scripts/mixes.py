@@ -58,6 +58,10 @@ class Runner:
         # two instances per tenant (self-pairs need distinct buffers)
         self.jobs = {t: [make_job(t, synth.preset(t, size, seed=11 + i), dev) for i in range(2)]
                      for t in tenants}
+        for js in self.jobs.values():   # bfs: depth + 1 level launches (one probe run)
+            for j in js:
+                if hasattr(j, "fit_levels"):
+                    j.fit_levels(self.acc)
         self.flush_buf = torch.empty(256 * 1024 * 1024 // 4, dtype=torch.float32, device=dev)
         self.ta = {}   # FAIR hints: isolated native times per tenant
 
