@@ -394,13 +394,10 @@ def run_rank(args, rank, world, local, ranks: Ranks) -> dict:
         flush_buf.fill_(1.0)
         torch.cuda.synchronize()
 
-    POL = {"fair": abi.POLICY_FAIR, "resolve": abi.POLICY_RESOLVE, "static": abi.POLICY_STATIC}
-    hints = {}   # FAIR: isolated-time profile per tenant (from the calibration below)
+    POL = {"resolve": abi.POLICY_RESOLVE, "static": abi.POLICY_STATIC}
     head_pol = POL[args.policy]
-    # reported beside the headline: STATIC (the paper's policy) and RESOLVE;
-    # FAIR (experimental) only with --all-policies
-    shown = POL if args.all_policies else ("static", "resolve")
-    other_pols = [p for p in shown if p != args.policy]
+    # reported beside the headline: STATIC (the paper's policy) and RESOLVE
+    other_pols = [p for p in POL if p != args.policy]
 
     def run_group(js, mode, e2e=False, launch_events=False, policy=None):
         policy = head_pol if policy is None else policy
@@ -408,8 +405,7 @@ def run_rank(args, rank, world, local, ranks: Ranks) -> dict:
             acc.set_mode(mode, policy)
         flush()
         acc.epoch()
-        iso = [hints.get(j.name, 0.0) for j in js] if policy == abi.POLICY_FAIR else None
-        ids = acc.submit(js, e2e=e2e, launch_events=launch_events, isolated_ms=iso)
+        ids = acc.submit(js, e2e=e2e, launch_events=launch_events)
         acc.sync()
         st = [acc.stats(i) for i in ids]
         lt = [acc.launch_times(i, j.launches()) for i, j in zip(ids, js)] if launch_events else None
@@ -451,7 +447,6 @@ def run_rank(args, rank, world, local, ranks: Ranks) -> dict:
             if mode == abi.MODE_SHARED:
                 iso_launch[j.name] = lts
     ta = [iso_native[t] for t in tenants]
-    hints.update(iso_native)
 
     def steps_loop(mode, k, e2e=False, policy=None):
         return [run_group(jobs, mode, e2e=e2e, launch_events=True, policy=policy) for _ in range(k)]
@@ -551,10 +546,9 @@ def main(argv=None):
     ap.add_argument("--config", default="c2", choices=["c1", "c2", "c5"])
     ap.add_argument("--impl", default="accel", choices=["accel", "reference"])
     ap.add_argument("--calib-reps", type=int, default=20)
-    ap.add_argument("--policy", default="resolve", choices=["fair", "resolve", "static"],
+    ap.add_argument("--policy", default="resolve", choices=["resolve", "static"],
                     help="SHARED-mode policy of the timed (headline) run; the others are reported too")
     ap.add_argument("--no-cpu-baseline", action="store_true")
-    ap.add_argument("--all-policies", action="store_true", help="also run the experimental FAIR policy")
     ap.add_argument("--out", default=None, help="also write the JSON line here")
     ap.add_argument("--hang-dump-s", type=float, default=0.0,
                     help="debug: dump every thread's Python stack after this many seconds")

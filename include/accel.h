@@ -51,19 +51,13 @@ typedef enum { ACCEL_MODE_NATIVE = 0, ACCEL_MODE_SHARED = 1 } accel_mode;
  * the resources initially allocated").  RESOLVE: quotas are recomputed on every
  * arrival and departure (BASELINE.json north star): shrinking lowers a live
  * quota word read at each dequeue, growing launches extra CTAs.
- * (Value 2 is retired: an SM-granular PARTITION policy was measured in round
- * 1 -- half the native throughput on C2 -- and removed.) */
-/* FAIR: RESOLVE whose weights follow the requests' measured slowdowns: the
- * monitor reads each running request's completed VGs every few hundred
- * microseconds, estimates its slowdown so far against its isolated time
- * (accel_request.isolated_ns, a profile the caller supplies) and re-solves
- * with weights growing with the slowdown, so laggards get a larger share
- * (§2.2, "changing the sharing ratio"; DESIGN.md
- * R-fair-1..3).  Requests without a hint keep the neutral weight. */
+ * (Values 2 and 3 are retired: an SM-granular PARTITION policy and a
+ * slowdown-feedback FAIR policy were measured in round 1 -- PARTITION at half
+ * the native throughput on C2, FAIR below RESOLVE on the sampled 4-mixes --
+ * and removed.) */
 typedef enum {
   ACCEL_POLICY_STATIC = 0,
-  ACCEL_POLICY_RESOLVE = 1,
-  ACCEL_POLICY_FAIR = 3
+  ACCEL_POLICY_RESOLVE = 1
 } accel_policy;
 
 #define ACCEL_ALL UINT64_MAX
@@ -117,6 +111,9 @@ typedef struct {
   int32_t regs;               /* regs/thread for the solver; 0 = query attrs   */
   uint32_t chunk;             /* VGs per dequeue (§6.4); 0 = default  */
   uint32_t args_size;         /* sizeof the kernel's argument struct           */
+  const void *order_fn;       /* host stub of accel_lpt_order<T>: the kernel's
+                                 dequeue-order cost model (T::vg_cost); NULL =
+                                 none (linear dequeue order)                    */
 } accel_kernel_desc;
 
 /* Fill *out with a built-in tenant kernel: "mop", "stencil", "histo", "bfs",
@@ -158,10 +155,14 @@ typedef struct {
   uint32_t repeat;       /* launches of this step, >= 1                          */
   const uint32_t *order_device; /* dequeue order (SHARED mode): the t-th VG handed out
                            is order_device[t], a permutation of 0..G-1 in device
-                           memory, caller-owned (e.g. most expensive VGs first, so
-                           that the cheapest ones form the tail); NULL = increasing
-                           linear order.  Static-grid kernels only.  NATIVE mode
-                           ignores it (hardware order).                            */
+                           memory, caller-owned; NULL = the kernel's own order:
+                           most expensive VGs first by its cost model when it has
+                           one (order_fn; G <= 8192), computed on the device by
+                           the library once per distinct (kernel, grid, args)
+                           and cached -- any permutation is correct, so a cached
+                           order only affects speed -- else increasing linear
+                           order.  Static-grid kernels only.  NATIVE mode ignores
+                           it (hardware order).                                    */
 } accel_launch;
 
 typedef struct { void *dst_device; int32_t value; uint64_t bytes; } accel_clear;
@@ -173,6 +174,8 @@ typedef struct { void *dst; const void *src; uint64_t bytes; } accel_copy; /* ho
 #define ACCEL_REQ_TRACE 2u          /* record one accel_vg_record per virtual group
                                        (accel_vg_trace); costs one %globaltimer
                                        pair and a 24-B store per VG */
+#define ACCEL_REQ_LINEAR_ORDER 4u   /* ignore the kernels' cost models: steps
+                                       without order_device dequeue linearly */
 
 typedef struct {
   int32_t tenant;             /* 0..ACCEL_MAX_TENANTS-1: selects the stream pair */
@@ -190,17 +193,6 @@ typedef struct {
   const accel_copy *h2d;
   uint32_t n_d2h;             /* device->host copies after the last launch      */
   const accel_copy *d2h;
-  uint64_t isolated_ns;       /* ACCEL_POLICY_FAIR: the request's isolated run
-                                 time (a profile); 0 = unknown (neutral weight) */
-  uint64_t vgs_hint;          /* FAIR: VGs the request will run; 0 = the sum of
-                                 its static grids (dynamic-total kernels such as
-                                 bfs run fewer: pass 0 AND isolated_ns = 0)     */
-  const float *progress_weights; /* FAIR, optional (HOST, copied at submit):
-                                 relative cost of the request's VGs in the order
-                                 they are dequeued (launch by launch, ticket
-                                 order), so that progress = cost share of the
-                                 VGs done rather than their count; NULL = equal */
-  uint64_t n_progress_weights; /* entries in progress_weights (== vgs_hint)     */
 } accel_request;
 
 /* Submit one request (solver run over the active set incl. this one).
@@ -267,6 +259,13 @@ typedef struct {
   uint32_t sm, cta;
 } accel_vg_record;
 int accel_vg_trace(accel_ctx *ctx, uint64_t request_id, accel_vg_record *out, uint64_t n, uint64_t *n_out);
+/* The dequeue order the library uses for a step of `kernel_id` over `grid`
+ * with `args` (accel_launch.order_device == NULL): VG ids by decreasing
+ * T::vg_cost, ties by increasing id (DESIGN.md R-disp-7), written to
+ * order_device[G] (DEVICE, caller-owned).  Synchronous.  ACCEL_EINVAL if the
+ * kernel has no cost model or G > 8192. */
+int accel_dequeue_order(accel_ctx *ctx, int32_t kernel_id, const accel_dim3 *grid, const void *args,
+                        uint32_t args_size, uint32_t *order_device);
 /* Forget completed requests (frees their descriptors); ACCEL_ALL = all done. */
 int accel_release(accel_ctx *ctx, uint64_t request_id);
 /* Streams of a tenant (cudaStream_t as void*), for interop (torch.cuda.ExternalStream). */
@@ -286,12 +285,6 @@ int accel_solve(const accel_caps *caps, const accel_demand *d, int32_t k, uint32
  * SHARED mode enqueues a group's grids in this order and the solver's
  * feasibility model F places them in it.  ACCEL_ENOFIT for an invalid demand. */
 int accel_placement_order(const accel_caps *caps, const accel_demand *d, int32_t k, int32_t *order_out);
-/* ACCEL_POLICY_FAIR weights (DESIGN.md R-fair-2): from the slowdowns so far
- * slowdown[k] (> 0; <= 0 = not yet known -> the neutral weight 16),
- * weight_out[i] = round(16 * (slowdown_i / g)^2) clamped to [1, 1024], g the
- * geometric mean of the known slowdowns. */
-int accel_fair_weights(const double *slowdown, int32_t k, uint32_t *weight_out);
-
 typedef struct {
   double unfairness;  /* max IS / min IS */
   double stp;         /* sum T(a)/T(s)                              */
@@ -308,6 +301,13 @@ int accel_metrics(const double *ta, const double *ts, int32_t k, accel_mix_metri
  * map from device memory the caller copies it to (64-B aligned). */
 int accel_tma_map_2d(void *out128, const void *gaddr, uint64_t inner, uint64_t outer,
                      uint64_t row_stride_bytes, uint32_t box_inner, uint32_t box_outer, int32_t swizzle);
+
+/* Encode a 3-D TMA tensor map (CUtensorMap) for a dense fp32 volume
+ * [d2][d1][d0] (d0 contiguous): row stride d0*4 and plane stride d0*d1*4
+ * bytes (both multiples of 16), box box0 x box1 x box2, no swizzle; boxes
+ * partly outside the volume read zeros.  Host only, like accel_tma_map_2d. */
+int accel_tma_map_3d(void *out128, const void *gaddr, uint64_t d0, uint64_t d1, uint64_t d2, uint32_t box0,
+                     uint32_t box1, uint32_t box2);
 
 /* Kernel execution overlap O = T(c)/T(t) of k
  * intervals [start[i], end[i]). */

@@ -15,7 +15,17 @@
 
 #ifdef __cplusplus
 extern "C" {
+#define ACCEL_ALIGN64 alignas(64)
+#else
+#define ACCEL_ALIGN64 _Alignas(64)
 #endif
+
+/* An encoded TMA tensor map (CUtensorMap, 128 B, 64-B aligned), see
+ * accel_tma_map_2d / accel_tma_map_3d.  Kernels that keep maps in their
+ * argument struct receive it as a __grid_constant__ kernel parameter. */
+typedef struct {
+  ACCEL_ALIGN64 uint8_t bytes[128];
+} accel_tmap;
 
 /* mop -- PAPER.md Fig. 8a (lines 735-746).  block 256, grid ceil(n/256).
  * out[g] = ina[g] + inb[g] if (g / 256) < nconst else ina[g] - inb[g]. */
@@ -42,6 +52,19 @@ typedef struct {
   uint32_t nx, ny, nz;
   float c0, c1;
 } accel_stencil_args;
+
+/* stencil_tma -- the same 7-point sweep (same launches, ping-pong and result
+ * buffer as "stencil"), nx % 4 == 0.  Planes staged by TMA: tmaps = 3-D maps
+ * (x, y, z extents nx, ny, nz; box 136 x 10 x 1; see accel_tma_map_3d) of a0,
+ * buf0 and buf1, in that order.  block 288 (8 consumer warps + 1 TMA producer
+ * warp), VG tile 128 x 8 x 8, grid (ceil(nx/128), ceil(ny/8), ceil(nz/8)). */
+typedef struct {
+  accel_tmap tmaps[3];
+  float *buf0;
+  float *buf1;
+  uint32_t nx, ny, nz;
+  float c0, c1;
+} accel_stencil_tma_args;
 
 /* histo -- saturating histogram (Parboil histo main + final fused).
  * block 256, VG = `per_vg` samples (multiple of 4096), grid ceil(n/per_vg).

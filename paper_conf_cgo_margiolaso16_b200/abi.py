@@ -23,12 +23,13 @@ ACCEL_ENOTREADY = -7
 ERRORS = {0: "ACCEL_OK", -1: "ACCEL_EINVAL", -2: "ACCEL_ENOFIT", -3: "ACCEL_ECUDA",
           -4: "ACCEL_ESTATE", -5: "ACCEL_ECOVERAGE", -6: "ACCEL_ENOMEM", -7: "ACCEL_ENOTREADY"}
 MODE_NATIVE, MODE_SHARED = 0, 1
-POLICY_STATIC, POLICY_RESOLVE, POLICY_FAIR = 0, 1, 3
+POLICY_STATIC, POLICY_RESOLVE = 0, 1
 ACCEL_ALL = 2**64 - 1
 MAX_TENANTS = 16
 MAX_STEPS = 8
 REQ_LAUNCH_EVENTS = 1
 REQ_TRACE = 2
+REQ_LINEAR_ORDER = 4
 
 u32, i32, u64, f32, f64, vp = C.c_uint32, C.c_int32, C.c_uint64, C.c_float, C.c_double, C.c_void_p
 
@@ -50,7 +51,7 @@ class accel_kernel_desc(C.Structure):
     _fields_ = [("name", C.c_char_p), ("persistent_fn", vp), ("persistent_resolve_fn", vp), ("native_fn", vp),
                 ("topup_fn", vp),
                 ("block", accel_dim3),
-                ("dyn_smem", u32), ("regs", i32), ("chunk", u32), ("args_size", u32)]
+                ("dyn_smem", u32), ("regs", i32), ("chunk", u32), ("args_size", u32), ("order_fn", vp)]
 
 
 class accel_kernel_info(C.Structure):
@@ -74,9 +75,7 @@ class accel_copy(C.Structure):
 class accel_request(C.Structure):
     _fields_ = [("tenant", i32), ("flags", u32), ("weight", u32), ("main_step", i32), ("n_steps", u32), ("steps", C.POINTER(accel_launch)),
                 ("n_clear", u32), ("clear", C.POINTER(accel_clear)), ("n_h2d", u32),
-                ("h2d", C.POINTER(accel_copy)), ("n_d2h", u32), ("d2h", C.POINTER(accel_copy)),
-                ("isolated_ns", u64), ("vgs_hint", u64),
-                ("progress_weights", vp), ("n_progress_weights", u64)]
+                ("h2d", C.POINTER(accel_copy)), ("n_d2h", u32), ("d2h", C.POINTER(accel_copy))]
 
 
 class accel_req_stats(C.Structure):
@@ -111,6 +110,13 @@ class accel_mop_args(C.Structure):
 class accel_stencil_args(C.Structure):
     _fields_ = [("a0", vp), ("buf0", vp), ("buf1", vp), ("nx", u32), ("ny", u32), ("nz", u32),
                 ("c0", f32), ("c1", f32)]
+
+
+class accel_stencil_tma_args(C.Structure):
+    # three 128-B CUtensorMaps first; the C struct is 64-B aligned, so its
+    # size is rounded up to a multiple of 64 (trailing pad)
+    _fields_ = [("tmaps", C.c_uint8 * 384), ("buf0", vp), ("buf1", vp), ("nx", u32), ("ny", u32), ("nz", u32),
+                ("c0", f32), ("c1", f32), ("_pad", C.c_uint8 * 28)]
 
 
 class accel_histo_args(C.Structure):
@@ -168,7 +174,7 @@ EXPORTS = [
     "accel_init", "accel_finalize", "accel_set_mode", "accel_last_error", "accel_builtin_kernel",
     "accel_builtin_count", "accel_builtin_name", "accel_kernel_register", "accel_kernel_info_get",
     "accel_submit", "accel_submit_group", "accel_sync", "accel_epoch", "accel_stats", "accel_release",
-    "accel_tenant_stream", "accel_launch_times", "accel_launch_stats", "accel_vg_trace", "accel_demand_of", "accel_solve", "accel_placement_order", "accel_fair_weights", "accel_metrics", "accel_overlap", "accel_tma_map_2d",
+    "accel_tenant_stream", "accel_launch_times", "accel_launch_stats", "accel_vg_trace", "accel_demand_of", "accel_solve", "accel_placement_order", "accel_dequeue_order", "accel_metrics", "accel_overlap", "accel_tma_map_2d", "accel_tma_map_3d",
 ]
 
 
@@ -207,10 +213,11 @@ def _load() -> C.CDLL:
         "accel_demand_of": (i32, [P(accel_caps), u32, u32, u32, u32, u32, P(accel_demand)]),
         "accel_solve": (i32, [P(accel_caps), P(accel_demand), i32, P(u32)]),
         "accel_placement_order": (i32, [P(accel_caps), P(accel_demand), i32, P(i32)]),
-        "accel_fair_weights": (i32, [P(f64), i32, P(u32)]),
+        "accel_dequeue_order": (i32, [vp, i32, P(accel_dim3), vp, u32, vp]),
         "accel_metrics": (i32, [P(f64), P(f64), i32, P(accel_mix_metrics)]),
         "accel_overlap": (i32, [P(f64), P(f64), i32, P(f64)]),
         "accel_tma_map_2d": (i32, [vp, vp, u64, u64, u64, u32, u32, i32]),
+        "accel_tma_map_3d": (i32, [vp, vp, u64, u64, u64, u32, u32, u32]),
     }
     for name, (res, args) in sig.items():
         fn = getattr(lib, name)
@@ -319,6 +326,13 @@ def accel_vg_trace(ctx, request_id: int):
     return arr
 
 
+def accel_dequeue_order(ctx, kernel_id: int, grid, args: C.Structure, order_device_ptr: int) -> None:
+    """The library's cost-model dequeue order for (kernel, grid, args) into a
+    device uint32 buffer of G entries (synchronous)."""
+    check(lib.accel_dequeue_order(ctx, kernel_id, C.byref(accel_dim3(*grid)), C.cast(C.pointer(args), C.c_void_p),
+                                  C.sizeof(args), C.c_void_p(order_device_ptr)), ctx)
+
+
 def accel_release(ctx, request_id: int = ACCEL_ALL) -> None:
     check(lib.accel_release(ctx, request_id), ctx)
 
@@ -353,12 +367,6 @@ def accel_placement_order(demands: list[accel_demand], caps: accel_caps | None =
     return list(out)[:k]
 
 
-def accel_fair_weights(slowdowns: list[float]) -> list[int]:
-    k = len(slowdowns)
-    out = (u32 * max(k, 1))()
-    check(lib.accel_fair_weights((f64 * max(k, 1))(*slowdowns), k, out))
-    return list(out)[:k]
-
 
 def accel_metrics(ta: list[float], ts: list[float]) -> accel_mix_metrics:
     k = len(ta)
@@ -371,6 +379,12 @@ def accel_tma_map_2d(gaddr: int, inner: int, outer: int, row_stride_bytes: int, 
                      box_outer: int, swizzle: int = 128) -> bytes:
     out = (C.c_ubyte * 128)()
     check(lib.accel_tma_map_2d(out, gaddr, inner, outer, row_stride_bytes, box_inner, box_outer, swizzle))
+    return bytes(out)
+
+
+def accel_tma_map_3d(gaddr: int, d0: int, d1: int, d2: int, box0: int, box1: int, box2: int) -> bytes:
+    out = (C.c_ubyte * 128)()
+    check(lib.accel_tma_map_3d(out, gaddr, d0, d1, d2, box0, box1, box2))
     return bytes(out)
 
 

@@ -41,8 +41,10 @@
 
 #include <cstdint>
 #include <type_traits>
+#include <utility>
 
 #include "accel.h"
+#include "../host/internal.h"
 
 namespace accel {
 
@@ -57,8 +59,7 @@ struct alignas(128) Ctl {
   uint32_t pad1[31];
   // ---- line 1
   uint32_t cur;       // highest request-relative launch index started (one red per launch)
-  uint32_t done_vgs;  // FAIR: VGs completed by the request (progress, read by the host monitor)
-  uint32_t pad2[30];
+  uint32_t pad2[31];
 };
 static_assert(sizeof(Ctl) == 256, "Ctl layout");
 
@@ -120,7 +121,7 @@ __device__ __forceinline__ void red_add_u32(uint32_t* p, uint32_t v) {
   asm volatile("red.relaxed.gpu.global.add.u32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
 }
 
-enum : uint32_t { kFlagStamps = 1u, kFlagAlive = 2u, kFlagProgress = 4u };
+enum : uint32_t { kFlagStamps = 1u, kFlagAlive = 2u };
 
 // Desc::qa = alive << 32 | next
 constexpr unsigned long long kAlive1 = 1ull << 32;
@@ -309,7 +310,6 @@ struct SchedState {
   uint32_t* coverage;
   accel_vg_record* trace;
   const uint32_t* order;   // dequeue order of the launch (nullptr: linear / spread)
-  uint32_t* progress;      // FAIR: Ctl::done_vgs (nullptr: not tracked)
   unsigned long long t0;   // trace: start of the current VG
   // RESOLVE, thread 0: view of the live quota and the admitted count, loaded
   // right after each dequeue and used at the next one, so the check adds no
@@ -476,7 +476,6 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     S->coverage = d->coverage;
     S->trace = d->trace;
     S->order = d->order;
-    S->progress = (d->flags & kFlagProgress) ? &d->ctl->done_vgs : nullptr;
     S->spread = has_spread<T>::value ? spread_factor(total) : 0u;
     S->prefetch_window = 2u * chunk * gridDim.x;
     S->template set_cur<has_spread<T>::value>(0, b);
@@ -512,7 +511,6 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     if (threadIdx.x == 0) {
       const uint32_t vg = S->cur[k].vg, id = S->cur[k].id;
       if (S->coverage != nullptr) atomicAdd(&S->coverage[id], 1u);
-      if (S->progress != nullptr) red_add_u32(S->progress, 1u);
       if (S->trace != nullptr) trace_vg(S->trace, id, S->t0, cta_tag);
       S->long_vg = globaltimer() - S->t0 > kLongVgNs;
       if (vg + 1 < S->end) {
@@ -545,7 +543,7 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
 // serves launch d.  cfg = chunk | kCfg* flags.  kResolve = RESOLVE policy.
 template <class T, bool kResolve>
 __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
-    accel_persistent(const typename T::Args args, Desc* __restrict__ d, uint32_t cfg) {
+    accel_persistent(const __grid_constant__ typename T::Args args, Desc* __restrict__ d, uint32_t cfg) {
   extern __shared__ __align__(128) char smem[];
   __shared__ SchedState S;
   serve<T, kResolve>(args, d, smem, &S, cfg, blockIdx.x);
@@ -556,7 +554,7 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
 // the step's later launches (each only once its predecessor completed).
 template <class T>
 __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
-    accel_topup(const typename T::Args args, Desc* __restrict__ d, uint32_t sticky) {
+    accel_topup(const __grid_constant__ typename T::Args args, Desc* __restrict__ d, uint32_t sticky) {
   extern __shared__ __align__(128) char smem[];
   __shared__ SchedState S;
   __shared__ uint32_t s_l;
@@ -584,10 +582,63 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
   }
 }
 
+// ---------------------------------------------------------------------------
+// Dequeue order from the tenant's cost model (DESIGN.md R-disp-7).  The
+// software queue may hand out VGs in any order; a
+// tenant with an optional
+//     static __device__ float vg_cost(const Args&, const VirtualBlock&);
+// (an estimate of a VG's work, e.g. the atoms a cutcp VG streams) gets its VGs
+// dealt most expensive first -- longest-processing-time-first list
+// scheduling over the persistent CTAs, so the tail after the queue runs dry
+// is short.  One CTA computes every cost and bitonic-sorts the keys
+// (~cost << 32 | vg: decreasing cost, ties by increasing id) in shared memory.
+template <class T, class = void>
+struct has_vg_cost : std::false_type {};
+template <class T>
+struct has_vg_cost<T, std::void_t<decltype(T::vg_cost(std::declval<const typename T::Args&>(),
+                                                      std::declval<const VirtualBlock&>()))>> : std::true_type {};
+
+
+template <class T>
+__global__ void __launch_bounds__(kOrderThreads) accel_lpt_order(const __grid_constant__ typename T::Args args, uint32_t gx,
+                                                                  uint32_t gy, uint32_t gz, uint32_t* order) {
+  extern __shared__ unsigned long long key[];
+  const uint32_t total = gx * gy * gz;
+  uint32_t n = 1;
+  while (n < total) n <<= 1;
+  for (uint32_t v = threadIdx.x; v < n; v += kOrderThreads) {
+    unsigned long long k = ~0ull;
+    if (v < total) {
+      const float c = fmaxf(T::vg_cost(args, decode(v, gx, gy, gz, 0)), 0.f);   // >= 0: bits are monotone
+      k = ((unsigned long long)(0xffffffffu - __float_as_uint(c)) << 32) | v;
+    }
+    key[v] = k;
+  }
+  __syncthreads();
+  for (uint32_t k = 2; k <= n; k <<= 1)
+    for (uint32_t j = k >> 1; j > 0; j >>= 1) {
+      for (uint32_t i = threadIdx.x; i < n; i += kOrderThreads) {
+        const uint32_t l = i ^ j;
+        if (l > i) {
+          const unsigned long long x = key[i], y = key[l];
+          if ((x > y) == ((i & k) == 0)) {
+            key[i] = y;
+            key[l] = x;
+          }
+        }
+      }
+      __syncthreads();
+    }
+  for (uint32_t v = threadIdx.x; v < total; v += kOrderThreads) order[v] = (uint32_t)key[v];
+}
+
 // The original kernel: one CTA per VG, hardware block scheduler (Fig. 1a).
+// (Every kernel takes the tenant's Args as a __grid_constant__ parameter: a
+// body may hand the address of a field to the TMA unit -- a CUtensorMap in
+// the argument struct, as stencil_tma does.)
 template <class T>
 __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
-    accel_native(const typename T::Args args, Desc* __restrict__ d, uint32_t /*unused*/) {
+    accel_native(const __grid_constant__ typename T::Args args, Desc* __restrict__ d, uint32_t /*unused*/) {
   extern __shared__ __align__(128) char smem[];
   const uint32_t flags = d->flags;
   if (threadIdx.x == 0 && (flags & kFlagStamps)) red_min_u64(&d->t_first, globaltimer());

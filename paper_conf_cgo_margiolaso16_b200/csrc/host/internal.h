@@ -41,6 +41,10 @@ cudaError_t launch_desc_init(const InitParams& p, uint32_t n_desc, cudaStream_t 
 // RESOLVE: wait (1 thread) until the request's last launch and its top-ups completed.
 cudaError_t launch_join(const Desc* last, cudaStream_t s);
 constexpr size_t kDescBytes = 384;
+// cost-model dequeue order (dispatch.cuh accel_lpt_order): one CTA sorts up to
+// kMaxOrderVGs 64-bit keys in dynamic shared memory
+constexpr uint32_t kMaxOrderVGs = 8192;
+constexpr uint32_t kOrderThreads = 512;
 constexpr size_t kCtlBytes = 256;
 
 }  // namespace accel

@@ -36,12 +36,8 @@ using accel::kDescBytes;
 
 constexpr uint32_t kPoolSlots = 16384;      // 4 MiB of descriptors
 constexpr uint32_t kFlagStamps = 1u, kFlagAlive = 2u;  // dispatch.cuh
-constexpr uint32_t kFlagProgress = 4u;     // dispatch.cuh: count completed VGs in Ctl::done_vgs
-constexpr int kFairPeriodUs = 150;         // FAIR: feedback period of the monitor
-constexpr double kFairW0 = 16.0;           // FAIR: neutral weight
-constexpr double kFairBeta = 2.0;          // FAIR: weight ~ (slowdown / geometric mean)^beta
 
-bool is_resolve(int policy) { return policy == ACCEL_POLICY_RESOLVE || policy == ACCEL_POLICY_FAIR; }
+bool is_resolve(int policy) { return policy == ACCEL_POLICY_RESOLVE; }
 
 struct Kernel {
   std::string name;
@@ -49,6 +45,7 @@ struct Kernel {
   const void* prfn;  // accel_persistent<T, RESOLVE>
   const void* nfn;
   const void* tfn;
+  const void* ofn;   // accel_lpt_order<T> (cost-model dequeue order), nullptr = none
   dim3 block;
   uint32_t dyn_smem;
   uint32_t chunk;
@@ -57,6 +54,14 @@ struct Kernel {
   int static_smem;
   int occ_p, occ_n;
   uint32_t threads() const { return block.x * block.y * block.z; }
+};
+
+// A cost-model dequeue order computed on the device (accel_lpt_order<T>) for
+// one (kernel, grid, args); `ready` once its kernel was enqueued (ev recorded).
+struct OrderEntry {
+  uint32_t* dev = nullptr;
+  cudaEvent_t ev = nullptr;
+  bool ready = false;
 };
 
 struct Step {
@@ -69,6 +74,7 @@ struct Step {
   uint32_t first;       // first descriptor (relative to the request's slot)
   uint64_t cov_offset;  // coverage offset of the first launch
   const uint32_t* order = nullptr;  // dequeue order (device), nullptr = linear
+  OrderEntry* order_entry = nullptr;  // library-computed order (cache entry)
 };
 
 struct Request {
@@ -103,12 +109,7 @@ struct Request {
   cudaEvent_t ev_early = nullptr;  // recorded after that launch (the main stream waits for it)
   uint32_t live = 0;         // RESOLVE: current live quota of the main step
   uint32_t provisioned = 0;  // RESOLVE: main-grid CTAs + sticky top-up CTAs
-  uint64_t iso_ns = 0;       // FAIR: isolated-time hint (0: none)
-  uint64_t vgs_hint = 0;     // FAIR: VGs the request runs
-  std::vector<double> cum_w; // FAIR: prefix sums of the progress weights (empty: count VGs)
-  cudaEvent_t ev_start = nullptr;  // FAIR: before the first launch (device-time elapsed)
   std::chrono::steady_clock::time_point t_submit;
-  uint32_t done_vgs = 0;     // FAIR: last progress read
   bool done = false;
   bool departed_seen = false;  // monitor already re-solved for this departure
   bool fetched = false;
@@ -169,7 +170,6 @@ struct accel_ctx {
   // of them must never share a stream: a pool with its own hardware queues
   // (16 main + 12 top-up + 1 control <= CUDA_DEVICE_MAX_CONNECTIONS = 32).
   uint32_t early_sms = 0;   // R-place-3: SMs held by early grids still waiting on the device
-  cudaEvent_t ev_now = nullptr;  // FAIR: "now" on the control stream
   static constexpr int kTopupStreams = 12;
   cudaStream_t topup[kTopupStreams] = {};
   // a growth grid is sticky (it follows its step's later launches), so a grid
@@ -196,10 +196,10 @@ struct accel_ctx {
   std::thread monitor;
   std::atomic<bool> stop{false};
   uint64_t monitor_solves = 0;
-  std::chrono::steady_clock::time_point last_fair{};
   uint32_t ablate = 0;   // env ACCEL_ABLATE: measurement-only cfg bits (dispatch.cuh kAbl*)
   std::vector<uint8_t> slot_used;
   std::map<uint64_t, std::unique_ptr<Request>> reqs;
+  std::map<std::string, OrderEntry> orders;   // cost-model orders by (kernel, grid, args)
   uint64_t next_id = 1;
   std::vector<cudaEvent_t> free_events;
 
@@ -323,6 +323,22 @@ int enqueue_begin(accel_ctx* ctx, Request* r) {
   CK(ctx, cudaEventRecord(r->ev_arrival, s));
   for (const accel_clear& c : r->clears) CK(ctx, cudaMemsetAsync(c.dst_device, c.value, c.bytes, s));
   for (const accel_copy& c : r->h2d) CK(ctx, cudaMemcpyAsync(c.dst, c.src, c.bytes, cudaMemcpyHostToDevice, s));
+  for (const Step& st : r->steps) {
+    OrderEntry* oe = st.order_entry;
+    if (oe == nullptr) continue;
+    if (!oe->ready) {   // first use: sort the VGs by the kernel's cost model on this stream
+      const Kernel& k = ctx->kernels[st.kid];
+      uint32_t gx = st.grid.x, gy = st.grid.y, gz = st.grid.z;
+      uint32_t* dst = oe->dev;
+      void* params[5] = {const_cast<unsigned char*>(st.args.data()), &gx, &gy, &gz, &dst};
+      CK(ctx, cudaLaunchKernel(k.ofn, dim3(1), dim3(accel::kOrderThreads), params,
+                               accel::kMaxOrderVGs * sizeof(unsigned long long), s));
+      CK(ctx, cudaEventRecord(oe->ev, s));
+      oe->ready = true;
+    } else {
+      CK(ctx, cudaStreamWaitEvent(s, oe->ev, 0));   // computed on another stream
+    }
+  }
   if (r->cov) CK(ctx, cudaMemsetAsync(r->cov, 0, r->cov_elems * sizeof(uint32_t), s));
   if (r->trace) CK(ctx, cudaMemsetAsync(r->trace, 0, r->trace_elems * sizeof(accel_vg_record), s));
   InitParams p{};
@@ -333,8 +349,7 @@ int enqueue_begin(accel_ctx* ctx, Request* r) {
   p.main_step = (uint32_t)r->main_step;
   p.coverage = r->cov;
   p.trace = r->trace;
-  p.flags = kFlagStamps | (shared ? kFlagAlive : 0u) |
-            (shared && ctx->cfg.policy == ACCEL_POLICY_FAIR && r->iso_ns ? kFlagProgress : 0u);
+  p.flags = kFlagStamps | (shared ? kFlagAlive : 0u);
   p.n_steps = (uint32_t)r->steps.size();
   for (size_t j = 0; j < r->steps.size(); ++j) {
     const Step& st = r->steps[j];
@@ -351,10 +366,6 @@ int enqueue_begin(accel_ctx* ctx, Request* r) {
   if (resolve) {
     CK(ctx, ctx->get_event(&r->ev_init));
     CK(ctx, cudaEventRecord(r->ev_init, s));
-  }
-  if (shared && ctx->cfg.policy == ACCEL_POLICY_FAIR && r->iso_ns) {
-    CK(ctx, ctx->get_event(&r->ev_start));
-    CK(ctx, cudaEventRecord(r->ev_start, s));
   }
   if (r->flags & ACCEL_REQ_LAUNCH_EVENTS) {
     r->ev_launch.resize(r->n_desc + 1);
@@ -499,9 +510,7 @@ int build_request(accel_ctx* ctx, const accel_request& in, std::unique_ptr<Reque
   r->flags = in.flags;
   r->weight = in.weight ? in.weight : 1;
   r->mode = ctx->cfg.mode;
-  r->iso_ns = in.isolated_ns;
   r->t_submit = std::chrono::steady_clock::now();
-  if (ctx->cfg.policy == ACCEL_POLICY_FAIR) r->weight = (uint32_t)kFairW0 * r->weight;  // neutral = W0
   uint32_t n_desc = 0;
   uint64_t cov = 0;
   if (in.main_step >= (int32_t)in.n_steps) return ctx->fail(ACCEL_EINVAL, "main_step out of range");
@@ -522,6 +531,19 @@ int build_request(accel_ctx* ctx, const accel_request& in, std::unique_ptr<Reque
     s.args.assign((const unsigned char*)L.args, (const unsigned char*)L.args + L.args_size);
     s.repeat = L.repeat;
     s.order = L.order_device;
+    if (!s.order && k.ofn && r->mode == ACCEL_MODE_SHARED && !(in.flags & ACCEL_REQ_LINEAR_ORDER) &&
+        total <= accel::kMaxOrderVGs) {
+      std::string key(reinterpret_cast<const char*>(&L.kernel_id), sizeof(L.kernel_id));
+      key.append(reinterpret_cast<const char*>(&L.grid), sizeof(L.grid));
+      key.append(s.args.begin(), s.args.end());
+      OrderEntry& oe = ctx->orders[key];
+      if (oe.dev == nullptr) {
+        CK(ctx, cudaMalloc(&oe.dev, total * sizeof(uint32_t)));
+        CK(ctx, cudaEventCreateWithFlags(&oe.ev, cudaEventDisableTiming));
+      }
+      s.order = oe.dev;
+      s.order_entry = &oe;
+    }
     s.quota = s.total;
     s.first = n_desc;
     s.cov_offset = cov;
@@ -531,17 +553,6 @@ int build_request(accel_ctx* ctx, const accel_request& in, std::unique_ptr<Reque
     if (in.main_step < 0 && r->steps.back().total > r->steps[r->main_step].total) r->main_step = (int)j;
   }
   r->n_desc = n_desc;
-  {
-    uint64_t vgs = 0;
-    for (const Step& s : r->steps) vgs += (uint64_t)s.total * s.repeat;
-    r->vgs_hint = in.vgs_hint ? in.vgs_hint : vgs;
-  }
-  if (in.progress_weights && in.n_progress_weights) {
-    r->cum_w.assign(in.n_progress_weights + 1, 0.0);
-    for (uint64_t i = 0; i < in.n_progress_weights; ++i)
-      r->cum_w[i + 1] = r->cum_w[i] + std::max(0.0, (double)in.progress_weights[i]);
-    if (!(r->cum_w.back() > 0.0)) r->cum_w.clear();
-  }
   r->cov_elems = ctx->cfg.verify ? cov : 0;
   r->trace_elems = (in.flags & ACCEL_REQ_TRACE) ? cov : 0;
   r->clears.assign(in.clear, in.clear + in.n_clear);
@@ -659,65 +670,6 @@ int assign_quotas(accel_ctx* ctx, std::vector<std::unique_ptr<Request>>& fresh) 
   return ACCEL_OK;
 }
 
-// FAIR (DESIGN.md R-fair-1..3): read every running request's completed VGs,
-// estimate its slowdown so far, sigma_i = elapsed_i / (progress_i * T_iso_i),
-// and set weight_i = W0 * (sigma_i / geomean sigma)^beta, clamped.  Returns
-// true when a weight moved by more than 25 % (then the caller re-solves).
-bool fair_weights(accel_ctx* ctx) {
-  std::vector<Request*> rs;
-  for (auto& kv : ctx->reqs) {
-    Request* r = kv.second.get();
-    if (r->mode == ACCEL_MODE_SHARED && !r->done && r->iso_ns && r->vgs_hint) rs.push_back(r);
-  }
-  if (rs.size() < 2) return false;
-  uint32_t* h = ctx->pinned_ring + (ctx->ring_pos % kRing);
-  ctx->ring_pos += (uint32_t)rs.size();
-  if (ctx->ring_pos % kRing < rs.size()) return false;  // wrap: skip this round
-  for (size_t i = 0; i < rs.size(); ++i)
-    if (ctx->cuda(cudaMemcpyAsync(h + i, ctx->ctl_pool + (size_t)rs[i]->slot * kCtlBytes + 132 /* Ctl::done_vgs */,
-                                  sizeof(uint32_t), cudaMemcpyDeviceToHost, ctx->ctl),
-                  "cudaMemcpyAsync(progress)"))
-      return false;
-  if (ctx->cuda(cudaEventRecord(ctx->ev_now, ctx->ctl), "cudaEventRecord(now)")) return false;
-  if (ctx->cuda(cudaStreamSynchronize(ctx->ctl), "cudaStreamSynchronize(ctl)")) return false;
-  std::vector<double> sig(rs.size(), 0.0);
-  int n = 0;
-  for (size_t i = 0; i < rs.size(); ++i) {
-    Request* r = rs[i];
-    r->done_vgs = h[i];
-    // elapsed device time since the request's first launch was reached on
-    // its stream (not host submission: copies and queueing are not progress)
-    if (!r->ev_start || cudaEventQuery(r->ev_start) != cudaSuccess) continue;
-    float el_ms = 0.f;
-    if (cudaEventElapsedTime(&el_ms, r->ev_start, ctx->ev_now) != cudaSuccess || el_ms <= 0.f) continue;
-    const double el = 1e6 * (double)el_ms;
-    // progress = cost share of the VGs done (progress_weights, in dequeue
-    // order), else their count
-    const double p = r->cum_w.empty()
-        ? std::min(1.0, (double)r->done_vgs / (double)r->vgs_hint)
-        : r->cum_w[std::min<size_t>(r->done_vgs, r->cum_w.size() - 1)] / r->cum_w.back();
-    if (p < 0.01 || el < 0.05 * (double)r->iso_ns) continue;  // too early to tell
-    sig[i] = el / (p * (double)r->iso_ns);
-    ++n;
-  }
-  if (n < 2) return false;
-  std::vector<uint32_t> w(rs.size());
-  accel_fair_weights(sig.data(), (int32_t)rs.size(), w.data());
-  bool moved = false;
-  for (size_t i = 0; i < rs.size(); ++i) {
-    if (sig[i] <= 0.0) continue;
-    const uint32_t wi = w[i];
-    if (wi * 4 > rs[i]->weight * 5 || wi * 5 < rs[i]->weight * 4) moved = true;
-    rs[i]->weight = wi;
-  }
-  if (moved && debug_on()) {
-    std::fprintf(stderr, "[accel] fair:");
-    for (size_t i = 0; i < rs.size(); ++i) std::fprintf(stderr, " t%d s=%.2f w=%u", rs[i]->tenant, sig[i], rs[i]->weight);
-    std::fprintf(stderr, "\n");
-  }
-  return moved;
-}
-
 // Host monitor (RESOLVE): detects departures without host synchronisation by
 // polling the requests' completion events, and re-solves the survivors.
 void monitor_loop(accel_ctx* ctx) {
@@ -743,15 +695,7 @@ void monitor_loop(accel_ctx* ctx) {
     }
     busy = running;
     if (departed && debug_on()) std::fprintf(stderr, "[accel] monitor: departure (running=%d)\n", (int)running);
-    bool resolve_now = departed && running;
-    if (running && ctx->cfg.policy == ACCEL_POLICY_FAIR) {
-      const auto now = std::chrono::steady_clock::now();
-      if (now - ctx->last_fair >= std::chrono::microseconds(kFairPeriodUs)) {
-        ctx->last_fair = now;
-        if (fair_weights(ctx)) resolve_now = true;
-      }
-    }
-    if (resolve_now) {
+    if (departed && running) {
       std::vector<std::unique_ptr<Request>> none;
       assign_quotas(ctx, none);
     }
@@ -823,7 +767,6 @@ void release_request(accel_ctx* ctx, Request* r) {
   if (r->trace) cudaFree(r->trace);
   if (r->ev_arrival) ctx->free_events.push_back(r->ev_arrival);
   if (r->ev_done) ctx->free_events.push_back(r->ev_done);
-  if (r->ev_start) ctx->free_events.push_back(r->ev_start);
   if (r->ev_early) ctx->free_events.push_back(r->ev_early);
   if (r->ev_init) ctx->free_events.push_back(r->ev_init);
   for (cudaEvent_t ev : r->ev_launch) ctx->free_events.push_back(ev);
@@ -834,29 +777,12 @@ void release_request(accel_ctx* ctx, Request* r) {
 
 extern "C" {
 
-int accel_fair_weights(const double* slowdown, int32_t k, uint32_t* weight_out) {
-  if (k < 0 || (k > 0 && (!slowdown || !weight_out))) return ACCEL_EINVAL;
-  double lsum = 0.0;
-  int n = 0;
-  for (int i = 0; i < k; ++i)
-    if (slowdown[i] > 0.0) {
-      lsum += std::log(slowdown[i]);
-      ++n;
-    }
-  const double gm = n ? std::exp(lsum / n) : 1.0;
-  for (int i = 0; i < k; ++i) {
-    const double w = slowdown[i] > 0.0 ? kFairW0 * std::pow(slowdown[i] / gm, kFairBeta) : kFairW0;
-    weight_out[i] = (uint32_t)std::lround(std::min(1024.0, std::max(1.0, w)));
-  }
-  return ACCEL_OK;
-}
-
 const char* accel_last_error(const accel_ctx* ctx) {
   return ctx ? ctx->err.c_str() : g_init_error.c_str();
 }
 
 bool policy_enabled(int32_t policy) {
-  return policy == ACCEL_POLICY_STATIC || policy == ACCEL_POLICY_RESOLVE || policy == ACCEL_POLICY_FAIR;
+  return policy == ACCEL_POLICY_STATIC || policy == ACCEL_POLICY_RESOLVE;
 }
 
 int accel_init(const accel_config* cfg, accel_ctx** out) {
@@ -887,7 +813,6 @@ int accel_init(const accel_config* cfg, accel_ctx** out) {
       return init_fail(e, "cudaStreamCreate");
   if ((e = cudaStreamCreateWithFlags(&ctx->ctl, cudaStreamNonBlocking)) != cudaSuccess)
     return init_fail(e, "cudaStreamCreate");
-  if ((e = cudaEventCreate(&ctx->ev_now)) != cudaSuccess) return init_fail(e, "cudaEventCreate");
   if ((e = cudaEventCreate(&ctx->epoch)) != cudaSuccess) return init_fail(e, "cudaEventCreate");
   if ((e = cudaMalloc(&ctx->pool, (size_t)kPoolSlots * kDescBytes)) != cudaSuccess)
     return init_fail(e, "cudaMalloc(pool)");
@@ -915,13 +840,17 @@ int accel_finalize(accel_ctx* ctx) {
     release_request(ctx, kv.second.get());
   }
   ctx->reqs.clear();
+  for (auto& kv : ctx->orders) {
+    if (kv.second.dev) cudaFree(kv.second.dev);
+    if (kv.second.ev) cudaEventDestroy(kv.second.ev);
+  }
+  ctx->orders.clear();
   for (cudaEvent_t ev : ctx->free_events) cudaEventDestroy(ev);
   for (int t = 0; t < ACCEL_MAX_TENANTS; ++t)
     if (ctx->main[t]) cudaStreamDestroy(ctx->main[t]);
   for (int t = 0; t < accel_ctx::kTopupStreams; ++t)
     if (ctx->topup[t]) cudaStreamDestroy(ctx->topup[t]);
   if (ctx->ctl) cudaStreamDestroy(ctx->ctl);
-  if (ctx->ev_now) cudaEventDestroy(ctx->ev_now);
   if (ctx->epoch) cudaEventDestroy(ctx->epoch);
   if (ctx->pool) cudaFree(ctx->pool);
   if (ctx->ctl_pool) cudaFree(ctx->ctl_pool);
@@ -958,6 +887,10 @@ int accel_kernel_register(accel_ctx* ctx, const accel_kernel_desc* d, int32_t* k
   k.prfn = d->persistent_resolve_fn ? d->persistent_resolve_fn : d->persistent_fn;
   k.nfn = d->native_fn;
   k.tfn = d->topup_fn ? d->topup_fn : d->persistent_fn;
+  k.ofn = d->order_fn;
+  if (k.ofn)
+    CK(ctx, cudaFuncSetAttribute(k.ofn, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                 (int)(accel::kMaxOrderVGs * sizeof(unsigned long long))));
   k.block = dim3(d->block.x, d->block.y ? d->block.y : 1, d->block.z ? d->block.z : 1);
   k.dyn_smem = d->dyn_smem;
   k.chunk = d->chunk ? d->chunk : 1;
@@ -1236,6 +1169,26 @@ int accel_vg_trace(accel_ctx* ctx, uint64_t request_id, accel_vg_record* out, ui
   const uint64_t m = std::min<uint64_t>(n, r->trace_elems);
   if (m) CK(ctx, cudaMemcpy(out, r->trace, m * sizeof(accel_vg_record), cudaMemcpyDeviceToHost));
   *n_out = r->trace_elems;
+  return ACCEL_OK;
+}
+
+int accel_dequeue_order(accel_ctx* ctx, int32_t kernel_id, const accel_dim3* grid, const void* args,
+                        uint32_t args_size, uint32_t* order_device) {
+  if (!ctx || !grid || !args || !order_device) return ACCEL_EINVAL;
+  std::lock_guard<std::mutex> g(ctx->mu);
+  if (ctx->poisoned) return ACCEL_ESTATE;
+  if (kernel_id < 0 || kernel_id >= (int)ctx->kernels.size()) return ctx->fail(ACCEL_EINVAL, "bad kernel_id");
+  const Kernel& k = ctx->kernels[kernel_id];
+  if (!k.ofn) return ctx->fail(ACCEL_EINVAL, k.name + " has no cost model");
+  if (args_size != k.args_size) return ctx->fail(ACCEL_EINVAL, "args_size mismatch for " + k.name);
+  const uint64_t total = (uint64_t)grid->x * grid->y * grid->z;
+  if (total == 0 || total > accel::kMaxOrderVGs) return ctx->fail(ACCEL_EINVAL, "grid too large for a cost order");
+  CK(ctx, cudaSetDevice(ctx->cfg.device));
+  uint32_t gx = grid->x, gy = grid->y, gz = grid->z;
+  void* params[5] = {const_cast<void*>(args), &gx, &gy, &gz, &order_device};
+  CK(ctx, cudaLaunchKernel(k.ofn, dim3(1), dim3(accel::kOrderThreads), params,
+                           accel::kMaxOrderVGs * sizeof(unsigned long long), ctx->ctl));
+  CK(ctx, cudaStreamSynchronize(ctx->ctl));
   return ACCEL_OK;
 }
 

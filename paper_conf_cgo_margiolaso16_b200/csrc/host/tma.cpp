@@ -48,3 +48,22 @@ extern "C" int accel_tma_map_2d(void* out128, const void* gaddr, uint64_t inner,
   std::memcpy(out128, &map, sizeof(map));
   return ACCEL_OK;
 }
+
+extern "C" int accel_tma_map_3d(void* out128, const void* gaddr, uint64_t d0, uint64_t d1, uint64_t d2,
+                                uint32_t box0, uint32_t box1, uint32_t box2) {
+  if (!out128 || !gaddr || !d0 || !d1 || !d2 || !box0 || !box1 || !box2) return ACCEL_EINVAL;
+  if ((d0 * 4) % 16 != 0) return ACCEL_EINVAL;
+  EncodeFn fn = encode_fn();
+  if (!fn) return ACCEL_ECUDA;
+  CUtensorMap map;
+  const cuuint64_t dims[3] = {d0, d1, d2};
+  const cuuint64_t strides[2] = {d0 * 4, d0 * d1 * 4};
+  const cuuint32_t box[3] = {box0, box1, box2};
+  const cuuint32_t estr[3] = {1, 1, 1};
+  CUresult r = fn(&map, CU_TENSOR_MAP_DATA_TYPE_FLOAT32, 3, const_cast<void*>(gaddr), dims, strides, box, estr,
+                  CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
+                  CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+  if (r != CUDA_SUCCESS) return ACCEL_EINVAL;
+  std::memcpy(out128, &map, sizeof(map));
+  return ACCEL_OK;
+}

@@ -16,6 +16,7 @@
 #include "tenants/sgemm_tc.cuh"
 #include "tenants/spmv.cuh"
 #include "tenants/stencil.cuh"
+#include "tenants/stencil_tma.cuh"
 #include "tenants/tpacf.cuh"
 
 namespace accel {
@@ -28,7 +29,6 @@ __global__ void desc_init_kernel(const InitParams p, uint32_t n_desc) {
   if (i == 0 && p.ctl != nullptr) {
     p.ctl->live = p.live_init;
     p.ctl->cur = 0;
-    p.ctl->done_vgs = 0;
   }
   if (i >= n_desc) return;
   uint32_t s = 0;
@@ -94,6 +94,10 @@ accel_kernel_desc make_desc(const char* name) {
   d.regs = 0;
   d.chunk = T::kChunk;
   d.args_size = sizeof(typename T::Args);
+  if constexpr (has_vg_cost<T>::value)
+    d.order_fn = reinterpret_cast<const void*>(&accel_lpt_order<T>);
+  else
+    d.order_fn = nullptr;
   return d;
 }
 
@@ -106,6 +110,7 @@ const Builtin kBuiltins[] = {
     {"mop", &make_desc<Mop>},
     {"stencil", &make_desc<Stencil>},
     {"stencil_x", &make_desc<StencilX>},
+    {"stencil_tma", &make_desc<StencilTma>},
     {"histo", &make_desc<Histo>},
     {"histo_wide", &make_desc<HistoWide>},
     {"bfs", &make_desc<Bfs>},

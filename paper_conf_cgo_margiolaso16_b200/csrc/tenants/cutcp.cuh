@@ -50,6 +50,34 @@ struct Cutcp {
     return fmaxf(0.f, fmaxf(clo - hi, lo - chi));
   }
 
+  // Dequeue-order cost model (dispatch.cuh accel_lpt_order): the atoms the
+  // body streams for this VG -- the same cell rows and trimmed x-ranges, in
+  // the same fp32 arithmetic.
+  static __device__ float vg_cost(const Args& a, const VirtualBlock& vb) {
+    const float h = a.h, cs = a.cell, cm = a.cutoff + 0.05f;
+    const int nc = (int)a.ncell;
+    const float bx0 = h * (float)(vb.x * 8), bx1 = h * (float)(vb.x * 8 + 7);
+    const float by0 = h * (float)(vb.y * 8), by1 = h * (float)(vb.y * 8 + 7);
+    const float bz0 = h * (float)(vb.z * 8), bz1 = h * (float)(vb.z * 8 + 7);
+    auto clampc = [&](int v) { return v < 0 ? 0 : (v >= nc ? nc - 1 : v); };
+    const int cy0 = clampc((int)floorf((by0 - cm) / cs)), cy1 = clampc((int)floorf((by1 + cm) / cs));
+    const int cz0 = clampc((int)floorf((bz0 - cm) / cs)), cz1 = clampc((int)floorf((bz1 + cm) / cs));
+    float atoms = 0.f;
+    for (int cz = cz0; cz <= cz1; ++cz) {
+      const float gz = gap(bz0, bz1, cz * cs, (cz + 1) * cs);
+      for (int cy = cy0; cy <= cy1; ++cy) {
+        const float gy = gap(by0, by1, cy * cs, (cy + 1) * cs);
+        const float d2 = gy * gy + gz * gz;
+        if (d2 >= cm * cm) continue;
+        const float rx = sqrtf(cm * cm - d2);
+        const int cx0 = clampc((int)floorf((bx0 - rx) / cs)), cx1 = clampc((int)floorf((bx1 + rx) / cs));
+        const int row = (cz * nc + cy) * nc;
+        atoms += (float)(a.cell_start[row + cx1 + 1] - a.cell_start[row + cx0]);
+      }
+    }
+    return atoms;
+  }
+
   static __device__ __forceinline__ void body(const Args& a, const VirtualBlock& vb, char* smem) {
     float4* tile = reinterpret_cast<float4*>(smem);
     const int t = threadIdx.x;

@@ -1,0 +1,149 @@
+// stencil_tma -- the 7-point Jacobi sweep of stencil.cuh with its planes
+// staged by the Tensor Memory Accelerator (PAPER.md names Parboil "stencil",
+// lines 290-291; BASELINE.json: "shared-memory or TMA staging for stencil").
+//
+// Why: stencil is the HBM-bound tenant of the Fig. 2 mix.  Under space
+// sharing it holds about a quarter of its solo CTAs, so its bandwidth is set
+// by the bytes in flight PER CTA, not by how many warps it has.  With cp.async
+// every byte in flight is a thread's outstanding copy and every plane a CTA
+// barrier; here one producer thread keeps kNS - 2 planes (~33 KB) in flight
+// per CTA through a ring of mbarrier-tracked TMA boxes, and the eight
+// consumer warps never meet at a CTA barrier inside a VG.
+//
+// VG = 128 x 8 x 8 (x, y, z) tile, 288 threads:
+//   warps 0..7  consumers: warp w owns row y0 + w, lane l owns x0+4l..x0+4l+3;
+//               the column z-1, z, z+1 lives in registers, y neighbours and
+//               the two x edges come from the staged plane, inner x
+//               neighbours from shuffles (same arithmetic and association as
+//               stencil.cuh, so the result is bit-identical)
+//   warp 8      producer (lane 0): plane p of the tile (z0 - 1 + p) is ONE
+//               cp.async.bulk.tensor.3d box (x0-4 .. x0+131, y0-1 .. y0+8, z)
+//               into ring slot p % kNS; boxes partly outside the volume read
+//               zeros (they only feed face cells, which copy the input)
+// Ring protocol: full[s] (1 arrival + the box's transaction bytes) and
+// empty[s] (one arrival per consumer warp once it last read the slot).  The
+// barriers are initialised per VG; every box a VG issues is waited for by
+// every consumer before the VG ends, so nothing asynchronous outlives it.
+// The tensor maps are __grid_constant__ kernel parameters (no descriptor in
+// global memory that a later job could overwrite).
+#pragma once
+#include "../device/dispatch.cuh"
+#include "accel_tenants.h"
+#include "tma.cuh"
+
+namespace accel {
+
+struct StencilTma {
+  using Args = accel_stencil_tma_args;
+  static constexpr int kConsumers = 8;
+  static constexpr int kThreads = 32 * (kConsumers + 1);
+  static constexpr int kTX = 128, kTY = 8, kTZ = 8;
+  static constexpr uint32_t kChunk = 1;
+#ifndef STENCIL_TMA_NS
+#define STENCIL_TMA_NS 8
+#endif
+  static constexpr int kNS = STENCIL_TMA_NS;            // ring slots (planes)
+  static constexpr int kMinBlocks = 5;
+  static constexpr int kRows = kTY + 2, kCols = kTX + 8;
+  static constexpr uint32_t kPlaneBytes = kRows * kCols * 4;          // 5440 (one box)
+  static constexpr uint32_t kSlot = (kPlaneBytes + 127) / 128 * 128;  // 5504
+  static constexpr uint32_t kDynSmem = kNS * kSlot + 2 * kNS * 8 + 128;   // + barriers, + alignment
+
+  static __device__ __forceinline__ void body(const Args& a, const VirtualBlock& vb, char* smem_raw) {
+    using namespace tma;
+    const uint32_t r = vb.launch_idx;
+    const int nx = (int)a.nx, ny = (int)a.ny, nz = (int)a.nz;
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    const int x0 = (int)vb.x * kTX, y0 = (int)vb.y * kTY, z0 = (int)vb.z * kTZ;
+    const int nzt = min(kTZ, nz - z0);
+    const int nplanes = nzt + 2;
+    const uint32_t sbase = (smem_u32(smem_raw) + 127u) & ~127u;
+    const uint32_t full0 = sbase + kNS * kSlot, empty0 = full0 + 8u * kNS;
+    auto slot = [&](int p) { return sbase + (uint32_t)(p % kNS) * kSlot; };
+    auto full = [&](int p) { return full0 + 8u * (uint32_t)(p % kNS); };
+    auto empty = [&](int p) { return empty0 + 8u * (uint32_t)(p % kNS); };
+    if (threadIdx.x == 0) {
+#pragma unroll
+      for (int q = 0; q < kNS; ++q) {
+        mbar_init(full0 + 8u * q, 1);
+        mbar_init(empty0 + 8u * q, kConsumers);
+      }
+      asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+    }
+    __syncthreads();
+
+    if (warp == kConsumers) {
+      // ---- producer: launch r reads a0 (r == 0), buf0 (r odd), buf1 (r even)
+      if (lane == 0) {
+        const accel_tmap* map = &a.tmaps[r == 0 ? 0 : ((r & 1u) ? 1 : 2)];
+        // the input was written through the generic proxy (by the previous
+        // launch, or -- for a RESOLVE top-up CTA -- by other CTAs of this
+        // grid, ordered by the dispatch's wait_complete and the barrier above)
+        asm volatile("fence.proxy.async.global;" ::: "memory");
+        for (int p = 0; p < nplanes; ++p) {
+          if (p >= kNS) mbar_wait(empty(p), (uint32_t)((p / kNS) - 1) & 1u);
+          mbar_expect_tx(full(p), kPlaneBytes);
+          tma_load_3d(slot(p), map, x0 - 4, y0 - 1, z0 - 1 + p, full(p));
+        }
+      }
+      return;   // (the dispatch loop's barrier follows)
+    }
+
+    // ---- consumers
+    float* __restrict__ out = (r & 1u) ? a.buf1 : a.buf0;
+    const int y = y0 + warp;
+    const bool active = x0 + 4 * lane < nx && y < ny;
+    const bool yint = y >= 1 && y <= ny - 2;
+    bool mxy[4];
+#pragma unroll
+    for (int e = 0; e < 4; ++e) {
+      const int x = x0 + 4 * lane + e;
+      mxy[e] = yint && x >= 1 && x <= nx - 2;
+    }
+    const float c0 = a.c0, c1 = a.c1;
+    const uint32_t own = 4u * (uint32_t)((warp + 1) * kCols + 4 + 4 * lane);
+    const uint32_t edge = 4u * (uint32_t)((warp + 1) * kCols + (lane == 31 ? 4 + kTX : 3));
+    mbar_wait(full(0), 0);
+    const float4 zm0 = lds_f4(slot(0) + own);
+    __syncwarp();
+    if (lane == 0) mbar_arrive(empty(0));      // plane z0-1 is only a z neighbour
+    mbar_wait(full(1), 0);
+    float4 zm = zm0, cur = lds_f4(slot(1) + own);
+    const long long pstr = (long long)nx * ny;
+    float* po = out + ((size_t)z0 * ny + y) * nx + x0 + 4 * lane;
+#pragma unroll 1
+    for (int i = 0; i < nzt; ++i) {
+      const int pz = i + 1;   // plane pz (= z0 + i) is `cur`
+      mbar_wait(full(pz + 1), (uint32_t)((pz + 1) / kNS) & 1u);
+      const uint32_t P = slot(pz);
+      const float4 zp = lds_f4(slot(pz + 1) + own);
+      const float4 ym = lds_f4(P + own - 4u * kCols);
+      const float4 yp = lds_f4(P + own + 4u * kCols);
+      const float ev = lds_f32(P + edge);
+      __syncwarp();
+      if (lane == 0) mbar_arrive(empty(pz));   // plane pz read for the last time
+      float xl = __shfl_up_sync(0xffffffffu, cur.w, 1);
+      float xr = __shfl_down_sync(0xffffffffu, cur.x, 1);
+      if (lane == 0) xl = ev;
+      if (lane == 31) xr = ev;
+      const int z = z0 + i;
+      float4 o = cur;
+      if (z >= 1 && z <= nz - 2) {   // uniform: z-face planes copy the input
+        const float vx = ((((((zm.x + zp.x) + ym.x) + yp.x) + xl) + cur.y) * c1 - cur.x * c0);
+        const float vy = ((((((zm.y + zp.y) + ym.y) + yp.y) + cur.x) + cur.z) * c1 - cur.y * c0);
+        const float vz = ((((((zm.z + zp.z) + ym.z) + yp.z) + cur.y) + cur.w) * c1 - cur.z * c0);
+        const float vw = ((((((zm.w + zp.w) + ym.w) + yp.w) + cur.z) + xr) * c1 - cur.w * c0);
+        if (mxy[0]) o.x = vx;
+        if (mxy[1]) o.y = vy;
+        if (mxy[2]) o.z = vz;
+        if (mxy[3]) o.w = vw;
+      }
+      if (active) *reinterpret_cast<float4*>(po) = o;
+      po += pstr;
+      zm = cur;
+      cur = zp;
+    }
+  }
+};
+
+}  // namespace accel

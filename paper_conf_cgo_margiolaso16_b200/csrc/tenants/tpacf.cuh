@@ -34,6 +34,13 @@ struct Tpacf {
   static constexpr uint32_t kDynSmem =
       kWarps * kMaxBins * 32 * sizeof(uint32_t) + kTile * sizeof(float4) + 32 * sizeof(float);
 
+  // Dequeue-order cost model (dispatch.cuh accel_lpt_order): Q tiles the VG
+  // walks -- DD / RR blocks (y <= S) start at their diagonal tile, DR blocks
+  // (y > S) walk all of them.
+  static __device__ float vg_cost(const Args& a, const VirtualBlock& vb) {
+    return vb.y <= a.nsets ? (float)vb.gx - (float)vb.x - 0.5f : (float)vb.gx;
+  }
+
   static __device__ __forceinline__ void body(const Args& a, const VirtualBlock& vb, char* smem) {
     uint32_t* hist = reinterpret_cast<uint32_t*>(smem);
     float4* qt = reinterpret_cast<float4*>(hist + kWarps * kMaxBins * 32);   // 16-B aligned (32 KB of counters)

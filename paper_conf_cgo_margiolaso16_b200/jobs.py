@@ -82,11 +82,6 @@ class Job:
         self._pinned_in: dict[str, torch.Tensor] = {}
         self._pinned_out: dict[str, torch.Tensor] = {}
         self.main_step = -1  # -1: the library picks the step with the most VGs
-        # FAIR policy: completed VGs / static VGs tracks progress (False for
-        # dynamic-total kernels, bfs: they run fewer VGs than their grids)
-        self.progress_hint = True
-        # FAIR: relative VG costs in dequeue order (None: every VG counts 1)
-        self.progress_weights: np.ndarray | None = None
 
     # ---- e2e: host buffers ----------------------------------------------
     def pin_host(self) -> None:
@@ -178,8 +173,11 @@ class MopJob(Job):
 
 class StencilJob(Job):
     TX, TY, TZ = 128, 8, 8
+    # nx % 4 == 0: TMA-staged planes ("stencil_tma", the default) or cp.async
+    # ("stencil"); any nx: "stencil_x"
+    KERNELS = ("stencil_tma", "stencil")
 
-    def __init__(self, d: dict, device="cuda"):
+    def __init__(self, d: dict, device="cuda", kernel: str | None = None):
         super().__init__(name="stencil", device=torch.device(device))
         self.nx, self.ny, self.nz, self.sweeps = d["nx"], d["ny"], d["nz"], d["sweeps"]
         n = self.nx * self.ny * self.nz
@@ -189,8 +187,18 @@ class StencilJob(Job):
         self.args = abi.accel_stencil_args(self.inputs["a0"].data_ptr(), self.buf[0].data_ptr(),
                                            self.buf[1].data_ptr(), self.nx, self.ny, self.nz, d["c0"], d["c1"])
         grid = (_cdiv(self.nx, self.TX), _cdiv(self.ny, self.TY), _cdiv(self.nz, self.TZ))
-        # rows 16-B aligned (nx % 4 == 0): cp.async 16-B pieces; else the any-nx kernel
-        self.steps = [Step("stencil" if self.nx % 4 == 0 else "stencil_x", grid, self.args, self.sweeps)]
+        kernel = kernel or d.get("kernel") or ("stencil_tma" if self.nx % 4 == 0 else "stencil_x")
+        if kernel != "stencil_x" and self.nx % 4:
+            raise ValueError(f"{kernel} needs nx % 4 == 0 (16-B rows); stencil_x takes any nx")
+        if kernel == "stencil_tma":
+            # 3-D maps of a0, buf0, buf1: box = one staged plane (136 x 10 x 1)
+            maps = b"".join(abi.accel_tma_map_3d(t.data_ptr(), self.nx, self.ny, self.nz, 136, 10, 1)
+                            for t in (self.inputs["a0"], self.buf[0], self.buf[1]))
+            self.args = abi.accel_stencil_tma_args((C.c_uint8 * 384).from_buffer_copy(maps), self.buf[0].data_ptr(),
+                                                   self.buf[1].data_ptr(), self.nx, self.ny, self.nz,
+                                                   d["c0"], d["c1"])
+        self.kernel = kernel
+        self.steps = [Step(kernel, grid, self.args, self.sweeps)]
 
     def result(self):
         return {"a": _np(self.out["a"], np.float32).reshape(self.nz, self.ny, self.nx)}
@@ -238,7 +246,6 @@ class BfsJob(Job):
 
     def __init__(self, d: dict, device="cuda", levels: int | None = None):
         super().__init__(name="bfs", device=torch.device(device))
-        self.progress_hint = False
         self.nv, self.ne, self.src = d["nv"], d["ne"], d["src"]
         self.levels = levels or d.get("levels", 24)
         self.inputs = {"row_ptr": _dev(d["row_ptr"], self.device), "col": _dev(d["col"], self.device)}
@@ -286,66 +293,6 @@ class BfsJob(Job):
         return {"bytes": b, "bytes_per_launch": b / self.levels, "bound": "hbm", "launches": self.levels}
 
 
-# ---- dequeue order (accel_launch.order_device): most expensive VGs first ----
-# The software queue hands out VGs in any order (DESIGN.md R-disp-7); ordering
-# them by decreasing estimated cost is longest-processing-time-first list
-# scheduling over the persistent CTAs: the last VGs dealt are the cheapest, so
-# the tail after the queue runs dry is short.  These are scheduling hints
-# computed from the inputs' shape, not results; NATIVE mode ignores them.
-def _lpt_order(cost: np.ndarray, device) -> torch.Tensor:
-    order = np.argsort(-np.asarray(cost, dtype=np.float64), kind="stable").astype(np.int32)
-    return torch.from_numpy(order).to(device)
-
-
-def _weights_in_order(cost: np.ndarray) -> np.ndarray:
-    """FAIR progress weights: the VG costs in the LPT dequeue order."""
-    c = np.asarray(cost, dtype=np.float64)
-    return np.ascontiguousarray(c[np.argsort(-c, kind="stable")], dtype=np.float32)
-
-
-def _cutcp_vg_cost(d: dict, grid) -> np.ndarray:
-    """Atoms a cutcp VG streams: the cell rows and trimmed x-ranges its body
-    walks (tenants/cutcp.cuh), counted from the cell index."""
-    gx, gy, gz = grid
-    h, cs, nc = float(d["h"]), float(d["cell"]), int(d["ncell_1d"])
-    cm = float(d["cutoff"]) + 0.05
-    cst = np.asarray(d["cell_start"], dtype=np.int64)
-    vx, vy, vz = np.meshgrid(np.arange(gx), np.arange(gy), np.arange(gz), indexing="xy")
-    vx, vy, vz = (a.transpose(2, 0, 1).ravel() for a in (vx, vy, vz))   # x fastest
-    b0 = [h * 8 * v for v in (vx, vy, vz)]
-    b1 = [h * (8 * v + 7) for v in (vx, vy, vz)]
-    cl = lambda v: np.clip(v, 0, nc - 1)  # noqa: E731
-    cy0, cy1 = cl(np.floor((b0[1] - cm) / cs).astype(int)), cl(np.floor((b1[1] + cm) / cs).astype(int))
-    cz0, cz1 = cl(np.floor((b0[2] - cm) / cs).astype(int)), cl(np.floor((b1[2] + cm) / cs).astype(int))
-    cost = np.zeros(vx.size)
-    gap = lambda lo, hi, c: np.maximum(0.0, np.maximum(c * cs - hi, lo - (c + 1) * cs))  # noqa: E731
-    for dz in range(int((cz1 - cz0).max()) + 1):
-        cz = cz0 + dz
-        okz = cz <= cz1
-        gzv = gap(b0[2], b1[2], cz)
-        for dy in range(int((cy1 - cy0).max()) + 1):
-            cy = cy0 + dy
-            ok = okz & (cy <= cy1)
-            gyv = gap(b0[1], b1[1], cy)
-            d2 = gyv * gyv + gzv * gzv
-            ok &= d2 < cm * cm
-            rx = np.sqrt(np.maximum(cm * cm - d2, 0.0))
-            cx0 = cl(np.floor((b0[0] - rx) / cs).astype(int))
-            cx1 = cl(np.floor((b1[0] + rx) / cs).astype(int))
-            row = (np.minimum(cz, nc - 1) * nc + np.minimum(cy, nc - 1)) * nc
-            cost += np.where(ok, cst[row + cx1 + 1] - cst[row + cx0], 0)
-    return cost
-
-
-def _tpacf_vg_cost(n: int, S: int, grid) -> np.ndarray:
-    """Q tiles a tpacf VG (x, y) walks: DD / RR blocks (y <= S) start at their
-    diagonal tile, DR blocks (y > S) walk all of them."""
-    gx, gy, _ = grid
-    x = np.tile(np.arange(gx), gy)
-    y = np.repeat(np.arange(gy), gx)
-    return np.where(y <= S, gx - x - 0.5, gx).astype(np.float64)
-
-
 class CutcpJob(Job):
     def __init__(self, d: dict, device="cuda"):
         super().__init__(name="cutcp", device=torch.device(device))
@@ -359,9 +306,8 @@ class CutcpJob(Job):
                                          d["ncell_1d"], d["cell"], self.nx, self.ny, self.nz, d["h"],
                                          d["cutoff"], d["excl"], self.v.data_ptr())
         grid = (_cdiv(self.nx, 8), _cdiv(self.ny, 8), _cdiv(self.nz, 8))
-        cost = _cutcp_vg_cost(d, grid)
-        self.steps = [Step("cutcp", grid, self.args, 1, _lpt_order(cost, self.device))]
-        self.progress_weights = _weights_in_order(cost)
+        # dequeue order: the library's cost model (Cutcp::vg_cost, most atoms first)
+        self.steps = [Step("cutcp", grid, self.args, 1)]
 
     def result(self):
         return {"v": _np(self.v, np.float32).reshape(self.nz, self.ny, self.nx)}
@@ -391,9 +337,8 @@ class TpacfJob(Job):
                                          p, p + 8 * nb, p + 16 * nb)
         self.clears = [(self.hists, 0)]
         grid = (_cdiv(self.n, 256), 2 * self.S + 1, 1)
-        cost = _tpacf_vg_cost(self.n, self.S, grid)
-        self.steps = [Step("tpacf", grid, self.args, 1, _lpt_order(cost, self.device))]
-        self.progress_weights = _weights_in_order(cost)
+        # dequeue order: the library's cost model (Tpacf::vg_cost, longest pair blocks first)
+        self.steps = [Step("tpacf", grid, self.args, 1)]
 
     def result(self):
         h = _np(self.hists, np.uint64).reshape(3, -1)

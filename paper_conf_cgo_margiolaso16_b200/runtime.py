@@ -58,20 +58,14 @@ class Accel:
 
     def submit(self, jobs: list[Job], tenants: list[int] | None = None, e2e: bool = False,
                weights: list[int] | None = None, launch_events: bool = False, trace: bool = False,
-               isolated_ms: list[float] | None = None) -> list[int]:
+               linear_order: bool = False) -> list[int]:
         """Submit jobs as one group arriving together, in list order.
         trace: record every virtual group (vg_trace)."""
         tenants = list(range(len(jobs))) if tenants is None else tenants
         weights = [1] * len(jobs) if weights is None else weights
-        fl = (abi.REQ_LAUNCH_EVENTS if launch_events else 0) | (abi.REQ_TRACE if trace else 0)
+        fl = ((abi.REQ_LAUNCH_EVENTS if launch_events else 0) | (abi.REQ_TRACE if trace else 0) |
+              (abi.REQ_LINEAR_ORDER if linear_order else 0))
         reqs = [j.request(self.kids, t, e2e, w, fl) for j, t, w in zip(jobs, tenants, weights)]
-        if isolated_ms is not None:   # FAIR policy: isolated-time profile per request
-            for r, j, ms in zip(reqs, jobs, isolated_ms):
-                r.isolated_ns = int(ms * 1e6) if (ms and j.progress_hint) else 0
-                if r.isolated_ns and j.progress_weights is not None:
-                    w = j.progress_weights   # kept alive by the job until submit returns
-                    r.progress_weights = w.ctypes.data
-                    r.n_progress_weights = len(w)
         # Job buffers (device inputs, tensor maps) were filled on torch's
         # stream; libaccel launches on its own non-blocking streams, which do
         # not order behind it.  Only torch's stream is waited on, never the

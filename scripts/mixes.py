@@ -42,8 +42,8 @@ from paper_conf_cgo_margiolaso16_b200.runtime import Accel  # noqa: E402
 
 TENANTS = ["bfs", "cutcp", "stencil", "tpacf", "histo", "spmv", "sgemm", "mriq"]
 MODES = [("native", abi.MODE_NATIVE, abi.POLICY_STATIC), ("resolve", abi.MODE_SHARED, abi.POLICY_RESOLVE),
-         ("static", abi.MODE_SHARED, abi.POLICY_STATIC), ("fair", abi.MODE_SHARED, abi.POLICY_FAIR)]
-SHARED = ["resolve", "static", "fair"]
+         ("static", abi.MODE_SHARED, abi.POLICY_STATIC)]
+SHARED = ["resolve", "static"]
 
 
 def gm(xs):
@@ -63,7 +63,6 @@ class Runner:
                 if hasattr(j, "fit_levels"):
                     j.fit_levels(self.acc)
         self.flush_buf = torch.empty(256 * 1024 * 1024 // 4, dtype=torch.float32, device=dev)
-        self.ta = {}   # FAIR hints: isolated native times per tenant
 
     def set(self, mode, policy):
         if self.acc.mode != mode or self.acc.policy != policy:
@@ -76,15 +75,14 @@ class Runner:
         torch.cuda.synchronize()
         self.acc.epoch()
         ids = []
-        iso = [self.ta.get(j.name, 0.0) for j in jobs] if policy == abi.POLICY_FAIR else None
         if delays_s is None:
-            ids = self.acc.submit(jobs, tenants=list(range(len(jobs))), isolated_ms=iso)
+            ids = self.acc.submit(jobs, tenants=list(range(len(jobs))))
         else:
             t0 = time.perf_counter()
             for i, (j, dl) in enumerate(zip(jobs, delays_s)):
                 while time.perf_counter() - t0 < dl:
                     pass
-                ids += self.acc.submit([j], tenants=[i], isolated_ms=None if iso is None else [iso[i]])
+                ids += self.acc.submit([j], tenants=[i])
         self.acc.sync()
         st = [self.acc.stats(i) for i in ids]
         self.acc.release()
@@ -216,7 +214,6 @@ def main():
         for _, mode, pol in MODES:
             r.run([j], mode, pol)
     ta = r.isolated(max(3, a.reps))
-    r.ta = dict(ta)
     print("T(a) ms", json.dumps({k: round(v, 3) for k, v in ta.items()}), flush=True)
     res = {"config": a.config, "size": a.size, "reps": a.reps, "T_a_ms": ta}
     if a.config == "c3":

@@ -8,7 +8,8 @@ and reports U, STP and ANTT per weight vector, beside NATIVE and the
 unweighted run.  Two families:
 
   rule   omega_i ~ T(a)_i ** alpha (a profile-guided rule, one alpha for every
-         mix: alpha = 0 is the paper's equal share)
+         mix: alpha = 0 is the paper's equal share, alpha < 0 favours the
+         shorter requests)
   grid   every vector in {1, 2, 3, 4}^K with min 1 (exhaustive: the best U
          reachable by static weights on this mix -- an upper bound on what a
          weight rule can do, NOT a policy)
@@ -48,6 +49,9 @@ def main():
     tenants, _, inputs = make_inputs(args.config, 0)
     jobs = [make_job(t, inputs[t], dev) for t in tenants]
     acc = Accel(device=0, mode=abi.MODE_SHARED)
+    for j in jobs:
+        if hasattr(j, "fit_levels"):
+            j.fit_levels(acc)
     flush_buf = torch.empty(256 * 1024 * 1024 // 4, dtype=torch.float32, device=dev)
 
     def run(js, mode, weights=None):
@@ -78,8 +82,10 @@ def main():
            "equal": measure(abi.MODE_SHARED), "rule": {}, "grid": []}
     print("native", res["native"])
     print("equal ", res["equal"])
-    for alpha in (0.25, 0.5, 0.75, 1.0):
-        w = [max(1, round(16 * (t / min(ta)) ** alpha)) for t in ta]
+    # alpha < 0: shorter requests get larger shares (shortest-first within the
+    # sharing); alpha > 0: longer ones do
+    for alpha in (-1.0, -0.75, -0.5, -0.25, 0.25, 0.5, 1.0):
+        w = [max(1, round(16 * (t / (min(ta) if alpha > 0 else max(ta))) ** alpha)) for t in ta]
         r = measure(abi.MODE_SHARED, w)
         r["weights"] = w
         res["rule"][str(alpha)] = r

@@ -120,34 +120,3 @@ def test_early_gemm_placement(racc, oracle_lib, partner):
         assert_close_fp32(jobs[1].result()["y"], oracle_lib.spmv(dp), what="spmv")
     # the GEMM kept its solved share: 74 CTAs (half the SMs) beside one partner
     assert st[0].quota_initial >= 37
-
-
-def test_fair_policy_mix_exact(oracle_lib):
-    """FAIR (R-fair-*): slowdown-feedback weights re-solve the quotas while the
-    requests run (progress counters, weighted by the LPT costs for cutcp and
-    tpacf); every VG still runs once and every result matches the oracle."""
-    import torch
-    if not torch.cuda.is_available():
-        pytest.skip("no GPU")
-    from paper_conf_cgo_margiolaso16_b200 import abi
-    from paper_conf_cgo_margiolaso16_b200.jobs import make_job
-    from paper_conf_cgo_margiolaso16_b200.runtime import Accel
-    ds = {"cutcp": synth.preset("cutcp", "default", seed=8),
-          "stencil": synth.preset("stencil", "default", seed=9, sweeps=40),
-          "tpacf": synth.preset("tpacf", "small", seed=10),
-          "histo": synth.preset("histo", "default", seed=11, iters=6)}
-    with Accel(device=0, mode=abi.MODE_SHARED, policy=abi.POLICY_FAIR, verify=True) as acc:
-        jobs = [make_job(n, d) for n, d in ds.items()]
-        # isolated-time hints far from the truth make the weights move
-        st = acc.run(jobs, isolated_ms=[0.3, 3.0, 0.2, 0.5])
-    assert all(s.coverage_ok == 1 for s in st)
-    r = np.random.Generator(np.random.PCG64(12))
-    dc = ds["cutcp"]
-    ijk = np.stack([r.integers(0, dc["nx"], 300), r.integers(0, dc["ny"], 300), r.integers(0, dc["nz"], 300)], 1)
-    v = jobs[0].result()["v"][ijk[:, 2], ijk[:, 1], ijk[:, 0]]
-    assert_close_fp32(v, oracle_lib.cutcp_points(dc, ijk), what="cutcp under FAIR")
-    assert_close_fp32(jobs[1].result()["a"][20:24], oracle_lib.stencil(ds["stencil"])[20:24], what="stencil under FAIR")
-    dd, rr, dr = oracle_lib.tpacf(ds["tpacf"])
-    t = jobs[2].result()
-    assert np.array_equal(t["dd"], dd) and np.array_equal(t["rr"], rr) and np.array_equal(t["dr"], dr)
-    assert np.array_equal(jobs[3].result()["counts"], oracle_lib.histo(ds["histo"])[0])

@@ -86,22 +86,29 @@ def test_mop_small_fullcaps(acc, oracle_lib):
                                        ("tiny", dict(nx=129, ny=8, nz=9, sweeps=2)),    # one column past a tile
                                        ("tiny", dict(nx=2, ny=5, nz=4, sweeps=2)),      # all faces
                                        ("small", dict(sweeps=10))])
-def test_stencil(acc_tiny_caps, oracle_lib, size, over):
+@pytest.mark.parametrize("kernel", ["default", "stencil"])
+def test_stencil(acc_tiny_caps, oracle_lib, size, over, kernel):
+    """default = stencil_tma (TMA ring) when nx % 4 == 0, stencil_x otherwise;
+    "stencil" = the cp.async staging (nx % 4 == 0 only)."""
     from paper_conf_cgo_margiolaso16_b200.jobs import StencilJob
     d = synth.preset("stencil", size, **over)
-    nat, sh, _ = run_modes(acc_tiny_caps, lambda: StencilJob(d))
+    if kernel == "stencil" and d["nx"] % 4:
+        pytest.skip("cp.async staging needs nx % 4 == 0")
+    k = None if kernel == "default" else kernel
+    nat, sh, _ = run_modes(acc_tiny_caps, lambda: StencilJob(d, kernel=k))
     same(nat, sh)
     assert_close_fp32(sh["a"], oracle_lib.stencil(d), what="stencil")
 
 
-def test_stencil_default_sampled(acc, oracle_lib):
+@pytest.mark.parametrize("kernel", ["stencil_tma", "stencil"])
+def test_stencil_default_sampled(acc, oracle_lib, kernel):
     """BASELINE size (512x512x64, 100 sweeps) in the bench's launch
     configuration; the oracle at full size is ~1.7e9 point-sweeps of plain C,
     so compare a handful of whole planes computed by the oracle on a z-slab
     that contains every point whose value can reach them (light cone)."""
     from paper_conf_cgo_margiolaso16_b200.jobs import StencilJob
     d = synth.preset("stencil", "default", sweeps=12)
-    job = StencilJob(d)
+    job = StencilJob(d, kernel=kernel)
     acc.run([job])
     got = job.result()["a"]
     # planes z in [20, 24): depend on z in [20-12, 24+12) only
@@ -194,7 +201,7 @@ def test_quota_matches_occupancy_for_single_tenant(acc):
     d = synth.preset("stencil", "default", sweeps=1)
     job = StencilJob(d)
     st = acc.run([job])[0]
-    info = acc.kernel_info("stencil")
+    info = acc.kernel_info(job.kernel)
     sms = torch.cuda.get_device_properties(0).multi_processor_count
     g = int(np.prod(job.steps[0].grid))
     assert st.quota_initial == min(g, sms * info.occ_persistent)

@@ -99,28 +99,6 @@ def test_metrics_equal():
         assert abi.accel_overlap(st, en) == pytest.approx(M.overlap(list(zip(st, en))), abs=1e-12)
 
 
-def test_fair_weights_closed_forms():
-    """FAIR weights (DESIGN.md R-fair-2): 16 * (s_i / geomean s)^2, clamped to
-    [1, 1024]; equal slowdowns -> equal (neutral) weights; unknown (<= 0) ->
-    neutral; doubling a slowdown quadruples the weight relative to the others."""
-    assert abi.accel_fair_weights([1.7, 1.7, 1.7, 1.7]) == [16] * 4
-    assert abi.accel_fair_weights([1.0, 2.0, 4.0]) == [4, 16, 64]
-    assert abi.accel_fair_weights([2.0, -1.0, 8.0]) == [4, 16, 64]
-    assert abi.accel_fair_weights([1.0, 1000.0]) == [1, 1024]
-    r = random.Random(9)
-    for _ in range(200):
-        s = [r.uniform(0.5, 6.0) for _ in range(r.randint(1, 8))]
-        w = abi.accel_fair_weights(s)
-        g = math.exp(sum(math.log(x) for x in s) / len(s))
-        assert w == [min(1024, max(1, round(16 * (x / g) ** 2))) for x in s] or all(
-            abs(a - b) <= 1 for a, b in zip(w, [16 * (x / g) ** 2 for x in s]))
-        # monotone: a larger slowdown never gets a smaller weight
-        for i in range(len(s)):
-            for j in range(len(s)):
-                if s[i] > s[j]:
-                    assert w[i] >= w[j]
-
-
 def test_placement_order_parity():
     """R-place-1: the library's enqueue / placement order equals the oracle's
     (largest per-CTA footprint first, ties in arrival order)."""
