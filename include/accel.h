@@ -293,6 +293,13 @@ typedef struct {
 } accel_mix_metrics;
 /* Sharing metrics of one mix from isolated times ta[k] and shared times ts[k]. */
 int accel_metrics(const double *ta, const double *ts, int32_t k, accel_mix_metrics *out);
+/* Weighted sharing (DESIGN.md R-metric-5; "changing
+ * the sharing ratio"): weighted slowdown WS_i = (ts_i / ta_i) * w_i / mean(w)
+ * -- equal for every request when the sharing honours the ratios w -- and the
+ * weighted unfairness max WS / min WS (= unfairness for equal weights).
+ * ws_out[k] may be NULL. */
+int accel_metrics_weighted(const double *ta, const double *ts, const double *w, int32_t k, double *wunfairness,
+                           double *ws_out);
 /* Encode a 2-D TMA tensor map (CUtensorMap, 128 B written to out128) for a
  * row-major fp32 matrix: `inner` elements per row (contiguous), `outer` rows,
  * rows row_stride_bytes apart (multiple of 16), box box_inner x box_outer,

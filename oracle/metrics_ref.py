@@ -8,6 +8,12 @@ PAPER.md §7.4 "Metrics" (lines 877-913), restated:
   speedup = T_baseline / T_X                   makespan ratio (901-908)
   STP, ANTT: named (911-913) but not printed; DESIGN.md R-metric-2 reads them
   as Eyerman & Eeckhout's STP = sum_i T(a)_i/T(s)_i, ANTT = mean_i T(s)_i/T(a)_i.
+Weighted sharing (DESIGN.md R-metric-5, "changing the
+sharing ratio"): request i is entitled to the share w_i / sum(w), so under
+weighted sharing its slowdown should scale as 1 / w_i; the weighted slowdown
+WS_i = IS_i * w_i / mean(w) is equal across requests when the sharing honours
+the ratios, and WU = max WS / min WS is the weighted unfairness (U when all
+weights are equal).
 Averages across mixes / request sizes are geometric means (R-metric-3: the
 printed 9.55x average of 6.8x, 10.4x, 12.27x is their geometric mean).
 """
@@ -37,6 +43,16 @@ def stp(ts: Sequence[float], ta: Sequence[float]) -> float:
 def antt(ts: Sequence[float], ta: Sequence[float]) -> float:
     IS = individual_slowdown(ts, ta)
     return sum(IS) / len(IS)
+
+
+def weighted_slowdown(ts: Sequence[float], ta: Sequence[float], w: Sequence[float]) -> list[float]:
+    wbar = sum(w) / len(w)
+    return [s / a * wi / wbar for s, a, wi in zip(ts, ta, w)]
+
+
+def weighted_unfairness(ts: Sequence[float], ta: Sequence[float], w: Sequence[float]) -> float:
+    ws = weighted_slowdown(ts, ta, w)
+    return max(ws) / min(ws)
 
 
 def throughput_speedup(makespan_baseline: float, makespan_x: float) -> float:

@@ -174,7 +174,7 @@ EXPORTS = [
     "accel_init", "accel_finalize", "accel_set_mode", "accel_last_error", "accel_builtin_kernel",
     "accel_builtin_count", "accel_builtin_name", "accel_kernel_register", "accel_kernel_info_get",
     "accel_submit", "accel_submit_group", "accel_sync", "accel_epoch", "accel_stats", "accel_release",
-    "accel_tenant_stream", "accel_launch_times", "accel_launch_stats", "accel_vg_trace", "accel_demand_of", "accel_solve", "accel_placement_order", "accel_dequeue_order", "accel_metrics", "accel_overlap", "accel_tma_map_2d", "accel_tma_map_3d",
+    "accel_tenant_stream", "accel_launch_times", "accel_launch_stats", "accel_vg_trace", "accel_demand_of", "accel_solve", "accel_placement_order", "accel_dequeue_order", "accel_metrics", "accel_metrics_weighted", "accel_overlap", "accel_tma_map_2d", "accel_tma_map_3d",
 ]
 
 
@@ -214,6 +214,7 @@ def _load() -> C.CDLL:
         "accel_solve": (i32, [P(accel_caps), P(accel_demand), i32, P(u32)]),
         "accel_placement_order": (i32, [P(accel_caps), P(accel_demand), i32, P(i32)]),
         "accel_dequeue_order": (i32, [vp, i32, P(accel_dim3), vp, u32, vp]),
+        "accel_metrics_weighted": (i32, [P(f64), P(f64), P(f64), i32, P(f64), P(f64)]),
         "accel_metrics": (i32, [P(f64), P(f64), i32, P(accel_mix_metrics)]),
         "accel_overlap": (i32, [P(f64), P(f64), i32, P(f64)]),
         "accel_tma_map_2d": (i32, [vp, vp, u64, u64, u64, u32, u32, i32]),
@@ -386,6 +387,16 @@ def accel_tma_map_3d(gaddr: int, d0: int, d1: int, d2: int, box0: int, box1: int
     out = (C.c_ubyte * 128)()
     check(lib.accel_tma_map_3d(out, gaddr, d0, d1, d2, box0, box1, box2))
     return bytes(out)
+
+
+def accel_metrics_weighted(ta: list[float], ts: list[float], w: list[float]) -> tuple[float, list[float]]:
+    """(weighted unfairness, weighted slowdowns) of one mix (DESIGN.md R-metric-5)."""
+    k = len(ta)
+    arr = lambda xs: (f64 * max(k, 1))(*xs)  # noqa: E731
+    wu = f64()
+    ws = (f64 * max(k, 1))()
+    check(lib.accel_metrics_weighted(arr(ta), arr(ts), arr(w), k, C.byref(wu), ws))
+    return wu.value, list(ws)[:k]
 
 
 def accel_overlap(start: list[float], end: list[float]) -> float:

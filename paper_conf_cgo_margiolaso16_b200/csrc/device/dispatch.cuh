@@ -538,6 +538,18 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
   if (threadIdx.x == 0) retire<kResolve>(d, cfg, S);
 }
 
+// Programmatic dependent launch (sm_90+): a request's launch l+1 is launched
+// with programmatic stream serialization after launch l (runtime.cpp).  Every
+// CTA lets the next grid launch as soon as it has started (once ALL CTAs of
+// this grid are resident, the next grid's CTAs may take the SM slots its
+// retiring CTAs free), then waits until the previous grid completed and its
+// writes are visible -- before it reads anything the previous launch wrote.
+// Launched without the attribute, both instructions are no-ops.
+__device__ __forceinline__ void pdl_enter() {
+  asm volatile("griddepcontrol.launch_dependents;" ::: "memory");
+  asm volatile("griddepcontrol.wait;" ::: "memory");
+}
+
 // -------------------------------------------------------------------------
 // The scheduling kernel: grid = quota (1-D), block = the original block;
 // serves launch d.  cfg = chunk | kCfg* flags.  kResolve = RESOLVE policy.
@@ -546,6 +558,7 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
     accel_persistent(const __grid_constant__ typename T::Args args, Desc* __restrict__ d, uint32_t cfg) {
   extern __shared__ __align__(128) char smem[];
   __shared__ SchedState S;
+  pdl_enter();
   serve<T, kResolve>(args, d, smem, &S, cfg, blockIdx.x);
 }
 
@@ -640,6 +653,7 @@ template <class T>
 __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
     accel_native(const __grid_constant__ typename T::Args args, Desc* __restrict__ d, uint32_t /*unused*/) {
   extern __shared__ __align__(128) char smem[];
+  pdl_enter();
   const uint32_t flags = d->flags;
   if (threadIdx.x == 0 && (flags & kFlagStamps)) red_min_u64(&d->t_first, globaltimer());
   VirtualBlock vb;

@@ -29,6 +29,26 @@ extern "C" int accel_metrics(const double* ta, const double* ts, int32_t k, acce
   return ACCEL_OK;
 }
 
+extern "C" int accel_metrics_weighted(const double* ta, const double* ts, const double* w, int32_t k,
+                                      double* wunfairness, double* ws_out) {
+  if (!ta || !ts || !w || !wunfairness || k <= 0) return ACCEL_EINVAL;
+  double wsum = 0.0;
+  for (int i = 0; i < k; ++i) {
+    if (!(ta[i] > 0.0) || !(ts[i] > 0.0) || !(w[i] > 0.0)) return ACCEL_EINVAL;
+    wsum += w[i];
+  }
+  const double wbar = wsum / k;
+  double mx = 0.0, mn = 0.0;
+  for (int i = 0; i < k; ++i) {
+    const double ws = ts[i] / ta[i] * w[i] / wbar;
+    if (ws_out) ws_out[i] = ws;
+    if (i == 0 || ws > mx) mx = ws;
+    if (i == 0 || ws < mn) mn = ws;
+  }
+  *wunfairness = mx / mn;
+  return ACCEL_OK;
+}
+
 extern "C" int accel_overlap(const double* start, const double* end, int32_t k, double* out) {
   if (!start || !end || !out || k <= 0) return ACCEL_EINVAL;
   std::vector<std::pair<double, double>> iv;

@@ -197,6 +197,7 @@ struct accel_ctx {
   std::atomic<bool> stop{false};
   uint64_t monitor_solves = 0;
   uint32_t ablate = 0;   // env ACCEL_ABLATE: measurement-only cfg bits (dispatch.cuh kAbl*)
+  bool pdl = true;       // programmatic dependent launch between a request's launches (env ACCEL_PDL=0: off)
   std::vector<uint8_t> slot_used;
   std::map<uint64_t, std::unique_ptr<Request>> reqs;
   std::map<std::string, OrderEntry> orders;   // cost-model orders by (kernel, grid, args)
@@ -438,7 +439,26 @@ int enqueue_next(accel_ctx* ctx, Request* r, bool* more) {
                    (1u << 19) | ctx->ablate;
     void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &cfg};
     const dim3 grid = shared ? dim3(st.quota, 1, 1) : dim3(st.grid.x, st.grid.y, st.grid.z);
-    CK(ctx, cudaLaunchKernel(shared ? (resolve ? k.prfn : k.pfn) : k.nfn, grid, k.block, params, k.dyn_smem, s));
+    const void* fn = shared ? (resolve ? k.prfn : k.pfn) : k.nfn;
+    if (li > 0 && ctx->pdl) {
+      // Programmatic dependent launch (both modes): launch l directly follows
+      // launch l-1 of the same request on this stream; its CTAs may become
+      // resident as l-1's CTAs retire and wait on the device
+      // (griddepcontrol.wait) instead of after a host-visible kernel boundary
+      cudaLaunchConfig_t lc = {};
+      lc.gridDim = grid;
+      lc.blockDim = k.block;
+      lc.dynamicSmemBytes = k.dyn_smem;
+      lc.stream = s;
+      cudaLaunchAttribute at[1];
+      at[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+      at[0].val.programmaticStreamSerializationAllowed = 1;
+      lc.attrs = at;
+      lc.numAttrs = 1;
+      CK(ctx, cudaLaunchKernelExC(&lc, fn, params));
+    } else {
+      CK(ctx, cudaLaunchKernel(fn, grid, k.block, params, k.dyn_smem, s));
+    }
     r->enq_li += 1;
     if (++r->enq_launch >= st.repeat) {
       r->enq_launch = 0;
@@ -823,6 +843,7 @@ int accel_init(const accel_config* cfg, accel_ctx** out) {
     return init_fail(e, "cudaHostAlloc(ring)");
   ctx->slot_used.assign(kPoolSlots, 0);
   if (const char* ab = std::getenv("ACCEL_ABLATE")) ctx->ablate = ((uint32_t)std::atoi(ab) & 31u) << 24;
+  if (const char* pd = std::getenv("ACCEL_PDL")) ctx->pdl = std::atoi(pd) != 0;
   accel_ctx* raw = ctx.release();
   raw->monitor = std::thread(monitor_loop, raw);
   *out = raw;

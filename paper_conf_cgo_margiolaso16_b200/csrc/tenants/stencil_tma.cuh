@@ -49,6 +49,13 @@ struct StencilTma {
   static constexpr uint32_t kSlot = (kPlaneBytes + 127) / 128 * 128;  // 5504
   static constexpr uint32_t kDynSmem = kNS * kSlot + 2 * kNS * 8 + 128;   // + barriers, + alignment
 
+  // ((((((zm + zp) + ym) + yp) + xm) + xp) * c1) - (c * c0), each step fp32 RN
+  static __device__ __forceinline__ float point(float zm, float zp, float ym, float yp, float xm, float xp, float c,
+                                                float c0, float c1) {
+    const float s = __fadd_rn(__fadd_rn(__fadd_rn(__fadd_rn(__fadd_rn(zm, zp), ym), yp), xm), xp);
+    return __fsub_rn(__fmul_rn(s, c1), __fmul_rn(c, c0));
+  }
+
   static __device__ __forceinline__ void body(const Args& a, const VirtualBlock& vb, char* smem_raw) {
     using namespace tma;
     const uint32_t r = vb.launch_idx;
@@ -129,10 +136,13 @@ struct StencilTma {
       const int z = z0 + i;
       float4 o = cur;
       if (z >= 1 && z <= nz - 2) {   // uniform: z-face planes copy the input
-        const float vx = ((((((zm.x + zp.x) + ym.x) + yp.x) + xl) + cur.y) * c1 - cur.x * c0);
-        const float vy = ((((((zm.y + zp.y) + ym.y) + yp.y) + cur.x) + cur.z) * c1 - cur.y * c0);
-        const float vz = ((((((zm.z + zp.z) + ym.z) + yp.z) + cur.y) + cur.w) * c1 - cur.z * c0);
-        const float vw = ((((((zm.w + zp.w) + ym.w) + yp.w) + cur.z) + xr) * c1 - cur.w * c0);
+        // fp32 round-to-nearest, this association, no FMA contraction: the
+        // compiler may contract a*c1 - b*c0 differently per instantiation
+        // (native vs persistent), which would break output transparency
+        const float vx = point(zm.x, zp.x, ym.x, yp.x, xl, cur.y, cur.x, c0, c1);
+        const float vy = point(zm.y, zp.y, ym.y, yp.y, cur.x, cur.z, cur.y, c0, c1);
+        const float vz = point(zm.z, zp.z, ym.z, yp.z, cur.y, cur.w, cur.z, c0, c1);
+        const float vw = point(zm.w, zp.w, ym.w, yp.w, cur.z, xr, cur.w, c0, c1);
         if (mxy[0]) o.x = vx;
         if (mxy[1]) o.y = vy;
         if (mxy[2]) o.z = vz;

@@ -56,7 +56,8 @@ class Runner:
         self.dev = dev
         self.acc = Accel(device=dev.index or 0, mode=abi.MODE_SHARED)
         # two instances per tenant (self-pairs need distinct buffers)
-        self.jobs = {t: [make_job(t, synth.preset(t, size, seed=11 + i), dev) for i in range(2)]
+        self.inputs = {t: synth.preset(t, size, seed=11) for t in tenants}
+        self.jobs = {t: [make_job(t, self.inputs[t], dev), make_job(t, synth.preset(t, size, seed=12), dev)]
                      for t in tenants}
         for js in self.jobs.values():   # bfs: depth + 1 level launches (one probe run)
             for j in js:
@@ -88,6 +89,17 @@ class Runner:
         self.acc.release()
         return st
 
+    def instance(self, t: str, i: int):
+        """The i-th instance of tenant t (its own buffers; mixes with repeated
+        tenants need one per occurrence).  Instances >= 2 reuse the inputs of
+        instance 0."""
+        while len(self.jobs[t]) <= i:
+            j = make_job(t, self.inputs[t], self.dev)
+            if hasattr(j, "fit_levels"):
+                j.fit_levels(self.acc)
+            self.jobs[t].append(j)
+        return self.jobs[t][i]
+
     def isolated(self, reps):
         ta = {}
         for t, (j, _) in self.jobs.items():
@@ -100,7 +112,8 @@ def mix_metrics(st, ta_list):
     ts = [s.elapsed_ms for s in st]
     m = abi.accel_metrics(ta_list, ts)
     mk = max(s.done_ms for s in st) - min(s.arrival_ms for s in st)
-    return {"U": m.unfairness, "STP": m.stp, "ANTT": m.antt, "makespan_ms": mk,
+    ov = abi.accel_overlap([float(s.first_start_ns) for s in st], [float(s.last_end_ns) for s in st])
+    return {"U": m.unfairness, "STP": m.stp, "ANTT": m.antt, "makespan_ms": mk, "O": ov,
             "WANTT": max(t / a for t, a in zip(ts, ta_list)), "ts_ms": ts}
 
 
@@ -153,18 +166,29 @@ def config4(r: Runner, ta, reps):
     return out
 
 
-def sampled(r: Runner, ta, reps, k, n, seed):
-    """n seeded random ordered k-tuples of distinct tenants,
-    submitted together; geometric means as in c3."""
+def sampled(r: Runner, ta, reps, k, n, seed, repeat=False):
+    """n seeded random ordered k-tuples of the tenants,
+    submitted together -- distinct tenants, or (repeat=True, the paper's
+    sampling space: ordered tuples with repetition)
+    any tenant any number of times, each occurrence its own instance;
+    geometric means as in c3."""
     g = np.random.Generator(np.random.PCG64(seed))
     mixes = []
+    keys = ("U", "STP", "ANTT", "makespan_ms", "WANTT", "O")
     for _ in range(n):
-        names = [TENANTS[i] for i in g.permutation(len(TENANTS))[:k]]
-        jobs = [r.jobs[t][0] for t in names]
+        if repeat:
+            names = [TENANTS[i] for i in g.integers(0, len(TENANTS), k)]
+        else:
+            names = [TENANTS[i] for i in g.permutation(len(TENANTS))[:k]]
+        seen: dict[str, int] = {}
+        jobs = []
+        for t in names:
+            jobs.append(r.instance(t, seen.get(t, 0)))
+            seen[t] = seen.get(t, 0) + 1
         res = {"mix": names}
         for name, mode, pol in MODES:
             runs = [mix_metrics(r.run(jobs, mode, pol), [ta[t] for t in names]) for _ in range(reps)]
-            res[name] = {kk: statistics.mean(x[kk] for x in runs) for kk in ("U", "STP", "ANTT", "makespan_ms", "WANTT")}
+            res[name] = {kk: statistics.mean(x[kk] for x in runs) for kk in keys}
         mixes.append(res)
         print(json.dumps({"mix": names, **{nm: {kk: round(v, 3) for kk, v in res[nm].items()} for nm, _, _ in MODES}}),
               flush=True)
@@ -178,13 +202,17 @@ def sampled(r: Runner, ta, reps, k, n, seed):
                      "throughput_speedup_gmean": gm([m["native"]["makespan_ms"] / m[name]["makespan_ms"]
                                                      for m in mixes]),
                      "WANTT_max": max(m[name]["WANTT"] for m in mixes),
+                     "ANTT_gmean": gm([m[name]["ANTT"] for m in mixes]),
+                     "O_mean": statistics.mean(m[name]["O"] for m in mixes),
                      # BASELINE.json target for 4-tenant mixes: U <= 1.5 and STP >= native
                      "target_met_pct": 100.0 * sum(m[name]["U"] <= 1.5 and m[name]["STP"] >= m["native"]["STP"]
                                                    for m in mixes) / len(mixes),
                      "U_le_1.5_pct": 100.0 * sum(m[name]["U"] <= 1.5 for m in mixes) / len(mixes),
                      "STP_ge_native_pct": 100.0 * sum(m[name]["STP"] >= m["native"]["STP"] for m in mixes) / len(mixes)}
     out["native"] = {"U_gmean": gm([m["native"]["U"] for m in mixes]),
-                     "WANTT_max": max(m["native"]["WANTT"] for m in mixes)}
+                     "WANTT_max": max(m["native"]["WANTT"] for m in mixes),
+                     "ANTT_gmean": gm([m["native"]["ANTT"] for m in mixes]),
+                     "O_mean": statistics.mean(m["native"]["O"] for m in mixes)}
     return mixes, out
 
 
@@ -194,6 +222,7 @@ def main():
     ap.add_argument("--k", type=int, default=4, help="f2: tenants per mix")
     ap.add_argument("--n", type=int, default=32, help="f2: number of sampled mixes")
     ap.add_argument("--seed", type=int, default=2024)
+    ap.add_argument("--repeat", action="store_true", help="f2: tuples with repetition (the paper's space)")
     ap.add_argument("--reps", type=int, default=3)
     ap.add_argument("--size", default="default")
     ap.add_argument("--out", default=None)
@@ -222,8 +251,8 @@ def main():
         res.update({"mixes": mixes, "summary": summ})
         print("SUMMARY", json.dumps(summ), flush=True)
     elif a.config == "f2":
-        mixes, summ = sampled(r, ta, a.reps, a.k, a.n, a.seed)
-        res.update({"mixes": mixes, "summary": summ, "k": a.k, "n": a.n, "seed": a.seed})
+        mixes, summ = sampled(r, ta, a.reps, a.k, a.n, a.seed, a.repeat)
+        res.update({"mixes": mixes, "summary": summ, "k": a.k, "n": a.n, "seed": a.seed, "repeat": a.repeat})
         print("SUMMARY", json.dumps(summ), flush=True)
     else:
         res["summary"] = config4(r, ta, a.reps)

@@ -120,3 +120,26 @@ def test_early_gemm_placement(racc, oracle_lib, partner):
         assert_close_fp32(jobs[1].result()["y"], oracle_lib.spmv(dp), what="spmv")
     # the GEMM kept its solved share: 74 CTAs (half the SMs) beside one partner
     assert st[0].quota_initial >= 37
+
+
+def test_explicit_weights_quotas_match_oracle():
+    """f1 ("changing the sharing ratio"): requests
+    submitted with explicit weights get exactly the quotas the oracle's
+    weighted solve gives (R-solver-7), and the results stay exact."""
+    import torch
+    from oracle import solver_ref as S
+    from paper_conf_cgo_margiolaso16_b200 import abi
+    from paper_conf_cgo_margiolaso16_b200.jobs import make_job
+    from paper_conf_cgo_margiolaso16_b200.runtime import Accel
+    n_sm = torch.cuda.get_device_properties(0).multi_processor_count
+    names = ["cutcp", "tpacf", "histo", "spmv"]
+    ds = {t: synth.preset(t, "small", seed=30 + i) for i, t in enumerate(names)}
+    for weights in ([1, 1, 1, 1], [3, 1, 1, 1], [1, 2, 4, 8]):
+        with Accel(device=0, mode=abi.MODE_SHARED, policy=abi.POLICY_STATIC, verify=True) as acc:
+            jobs = [make_job(t, ds[t]) for t in names]
+            st = acc.run(jobs, weights=weights)
+            infos = [acc.kernel_info(j.steps[j.main_step].kernel) for j in jobs]
+        assert all(s.coverage_ok == 1 for s in st)
+        dem = [S.Demand(i.thr, i.regs, i.smem, i.cta, int(np.prod(j.steps[j.main_step].grid)), w)
+               for i, j, w in zip(infos, jobs, weights)]
+        assert [s.quota_initial for s in st] == S.solve(dem, S.Caps(sms=n_sm)), weights

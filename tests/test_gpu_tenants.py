@@ -303,3 +303,35 @@ def test_config2_fig2_mix(acc, oracle_lib):
         if mode == abi.MODE_SHARED:
             assert len({s.quota_initial for s in st}) >= 1
     acc.set_mode(abi.MODE_SHARED)
+
+
+def _stencil_fp32_replica(d):
+    """numpy float32 with the kernels' association ("numpy
+    float32 with the same parenthesisation reproduces the result exactly"):
+    ((((((zm + zp) + ym) + yp) + xm) + xp) * c1) - (a * c0), faces copy."""
+    a = d["a0"].reshape(d["nz"], d["ny"], d["nx"]).astype(np.float32)
+    c0, c1 = np.float32(d["c0"]), np.float32(d["c1"])
+    for _ in range(d["sweeps"]):
+        o = a.copy()
+        s = a[:-2, 1:-1, 1:-1] + a[2:, 1:-1, 1:-1]
+        s = s + a[1:-1, :-2, 1:-1]
+        s = s + a[1:-1, 2:, 1:-1]
+        s = s + a[1:-1, 1:-1, :-2]
+        s = s + a[1:-1, 1:-1, 2:]
+        o[1:-1, 1:-1, 1:-1] = s * c1 - a[1:-1, 1:-1, 1:-1] * c0
+        a = o
+    return a
+
+
+@pytest.mark.parametrize("kernel,over", [("stencil_tma", dict(nx=136, ny=17, nz=19, sweeps=4)),
+                                         ("stencil", dict(nx=136, ny=17, nz=19, sweeps=4)),
+                                         ("stencil_x", dict(nx=70, ny=21, nz=19, sweeps=3))])
+def test_stencil_bit_exact_fp32_sequence(acc_tiny_caps, kernel, over):
+    """Every stencil kernel computes the pinned fp32 round-to-nearest sequence
+    (no FMA contraction), so native, persistent and a numpy float32 replica
+    agree bit for bit."""
+    from paper_conf_cgo_margiolaso16_b200.jobs import StencilJob
+    d = synth.preset("stencil", "tiny", **over)
+    nat, sh, _ = run_modes(acc_tiny_caps, lambda: StencilJob(d, kernel=kernel))
+    ref = _stencil_fp32_replica(d)
+    assert np.array_equal(nat["a"], ref) and np.array_equal(sh["a"], ref)

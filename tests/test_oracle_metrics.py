@@ -90,3 +90,31 @@ def test_geomean_closed_form():
     assert M.geomean([3.0]) == pytest.approx(3.0)
     assert M.geomean([10.0, 0.1]) == pytest.approx(1.0)
     assert math.isclose(M.geomean([1.5] * 7), 1.5)
+
+
+# ---- weighted sharing (DESIGN.md R-metric-5) --------
+
+def test_weighted_unfairness_equal_weights_is_unfairness():
+    ta, ts = [1.0, 2.0, 0.5], [3.0, 2.5, 2.0]
+    for w in ([1, 1, 1], [7, 7, 7]):
+        assert M.weighted_unfairness(ts, ta, w) == pytest.approx(M.unfairness(ts, ta))
+
+
+def test_weighted_unfairness_honoured_ratio_is_one():
+    """Two equal jobs, ratio 2:1.  Weighted processor sharing on a fluid
+    device: A (weight 2) runs at 2/3 of the device until it finishes at 1.5,
+    B at 1/3 until then (0.5 done) and alone after (done at 2.0): IS = 1.5 and
+    2.0 -- the LATER job is still favoured less than 2x because B runs alone
+    at the end.  WU is the measure: with the ratio honoured throughout (both
+    finish in proportion, IS = 1.5 and 3), WS = 1.5*2/1.5 = 2 = 3*1/1.5."""
+    assert M.weighted_unfairness([1.5, 3.0], [1.0, 1.0], [2, 1]) == pytest.approx(1.0)
+    assert M.weighted_slowdown([1.5, 3.0], [1.0, 1.0], [2, 1]) == pytest.approx([2.0, 2.0])
+    # the fluid schedule above is not weighted-fair: WS = [2, 4/3]
+    assert M.weighted_unfairness([1.5, 2.0], [1.0, 1.0], [2, 1]) == pytest.approx(1.5)
+
+
+def test_weighted_unfairness_scale_invariant():
+    ta, ts, w = [1.0, 2.0, 4.0], [2.0, 5.0, 6.0], [1.0, 3.0, 2.0]
+    a = M.weighted_unfairness(ts, ta, w)
+    assert M.weighted_unfairness(ts, ta, [10 * x for x in w]) == pytest.approx(a)
+    assert M.weighted_unfairness([3 * x for x in ts], ta, w) == pytest.approx(a)

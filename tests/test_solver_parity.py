@@ -111,3 +111,16 @@ def test_placement_order_parity():
     g, sp = S.demand_of(640, 96, 189 * 1024, 512), S.demand_of(256, 40, 0, 2304)
     assert S.placement_order([sp, g]) == [1, 0]
     assert abi.accel_placement_order([_to_c(sp), _to_c(g)]) == [1, 0]
+
+
+def test_weighted_metrics_equal():
+    """libaccel accel_metrics_weighted == oracle/metrics_ref (R-metric-5)."""
+    r = random.Random(9)
+    for _ in range(300):
+        k = r.randint(1, 8)
+        ta = [r.uniform(0.1, 5) for _ in range(k)]
+        ts = [a * r.uniform(1, 6) for a in ta]
+        w = [r.choice([1, 2, 3, 16, 0.5]) for _ in range(k)]
+        wu, ws = abi.accel_metrics_weighted(ta, ts, w)
+        assert wu == pytest.approx(M.weighted_unfairness(ts, ta, w), rel=1e-12)
+        assert ws == pytest.approx(M.weighted_slowdown(ts, ta, w), rel=1e-12)
