@@ -64,6 +64,8 @@ typedef struct {
   float *buf1;
   uint32_t nx, ny, nz;
   float c0, c1;
+  const accel_tmap *gmaps;  /* diagnostic: non-NULL = read the three maps from
+                               this DEVICE array instead of the parameters */
 } accel_stencil_tma_args;
 
 /* histo -- saturating histogram (Parboil histo main + final fused).

@@ -18,6 +18,9 @@ ROOT = os.path.dirname(PKG)
 CSRC = os.path.join(PKG, "csrc")
 INCLUDE = os.path.join(ROOT, "include")
 LIB = os.path.join(PKG, "libaccel.so")
+LIB_RT = os.path.join(PKG, "libaccel_rt.so")             # same objects, shared CUDA runtime
+LIB_INTERCEPT = os.path.join(PKG, "libaccel_intercept.so")
+APP = os.path.join(ROOT, "examples", "intercept_app")
 NVCC = os.environ.get("NVCC", "/usr/local/cuda/bin/nvcc")
 ARCH = ["-gencode", "arch=compute_100a,code=sm_100a"]
 FLAGS = ["-O3", "-lineinfo", "-std=c++17", "-Xcompiler", "-fPIC,-O3", "--expt-relaxed-constexpr",
@@ -31,13 +34,16 @@ def sources() -> list[str]:
 def deps() -> list[str]:
     pats = ["*.cu", "*.cuh", "*.h", "*.cpp", "*/*.cu", "*/*.cuh", "*/*.h", "*/*.cpp"]
     out = [p for pat in pats for p in glob.glob(os.path.join(CSRC, pat))]
-    return out + glob.glob(os.path.join(INCLUDE, "*.h"))
+    return out + glob.glob(os.path.join(INCLUDE, "*.h")) + glob.glob(os.path.join(INCLUDE, "*.cuh")) + \
+        glob.glob(os.path.join(ROOT, "examples", "*.cu"))
 
 
 def up_to_date() -> bool:
     if not os.path.exists(LIB):
         return False
     t = os.path.getmtime(LIB)
+    if not all(os.path.exists(p) for p in (LIB_RT, LIB_INTERCEPT)):
+        return False
     return all(os.path.getmtime(p) <= t for p in deps())
 
 
@@ -58,7 +64,30 @@ def build(force: bool = False, verbose: bool = False) -> str:
     subprocess.check_call([NVCC, *ARCH, "-shared", "-cudart", "static", "-o", tmp, *objs,
                            "-Xcompiler", "-fPIC"])
     os.replace(tmp, LIB)
+    build_intercept(objs)
     return LIB
+
+
+def build_intercept(objs: list[str]) -> None:
+    """Transparent interception: the same objects linked
+    against the SHARED CUDA runtime (libaccel_rt.so: an application's kernel
+    stubs and the library must live in one runtime instance), the LD_PRELOAD
+    shim over cudaLaunchKernel (libaccel_intercept.so), and the example
+    application (examples/intercept_app, shared runtime)."""
+    tmp = LIB_RT + f".tmp{os.getpid()}"
+    subprocess.check_call([NVCC, *ARCH, "-shared", "-cudart", "shared", "-o", tmp, *objs, "-Xcompiler", "-fPIC"])
+    os.replace(tmp, LIB_RT)
+    tmp = LIB_INTERCEPT + f".tmp{os.getpid()}"
+    subprocess.check_call([NVCC, "-std=c++17", "-O2", "-shared", "-cudart", "shared", "-Xcompiler", "-fPIC",
+                           "-I", INCLUDE, os.path.join(CSRC, "intercept", "intercept.cpp"), "-o", tmp,
+                           "-L", PKG, "-laccel_rt", "-ldl", "-Xlinker", "-rpath,$ORIGIN"])
+    os.replace(tmp, LIB_INTERCEPT)
+    app_src = os.path.join(ROOT, "examples", "intercept_app.cu")
+    if os.path.exists(app_src):
+        tmp = APP + f".tmp{os.getpid()}"
+        subprocess.check_call([NVCC, *ARCH, "-O2", "-std=c++17", "--expt-relaxed-constexpr", "-cudart", "shared",
+                               "-I", INCLUDE, "-I", CSRC, app_src, "-o", tmp])
+        os.replace(tmp, APP)
 
 
 if __name__ == "__main__":

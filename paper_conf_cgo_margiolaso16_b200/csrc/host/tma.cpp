@@ -5,6 +5,7 @@
 #include <cuda.h>
 #include <cuda_runtime.h>
 
+#include <cstdlib>
 #include <cstring>
 
 #include "accel.h"
@@ -60,9 +61,12 @@ extern "C" int accel_tma_map_3d(void* out128, const void* gaddr, uint64_t d0, ui
   const cuuint64_t strides[2] = {d0 * 4, d0 * d1 * 4};
   const cuuint32_t box[3] = {box0, box1, box2};
   const cuuint32_t estr[3] = {1, 1, 1};
+  // diagnostic knob (scripts/diag_tma.py): L2 promotion of the boxes
+  CUtensorMapL2promotion promo = CU_TENSOR_MAP_L2_PROMOTION_L2_256B;
+  if (const char* e = std::getenv("ACCEL_TMA_PROMO"))
+    promo = static_cast<CUtensorMapL2promotion>(std::atoi(e) & 3);
   CUresult r = fn(&map, CU_TENSOR_MAP_DATA_TYPE_FLOAT32, 3, const_cast<void*>(gaddr), dims, strides, box, estr,
-                  CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
-                  CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+                  CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, promo, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
   if (r != CUDA_SUCCESS) return ACCEL_EINVAL;
   std::memcpy(out128, &map, sizeof(map));
   return ACCEL_OK;

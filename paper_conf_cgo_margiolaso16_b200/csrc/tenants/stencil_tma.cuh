@@ -82,7 +82,9 @@ struct StencilTma {
     if (warp == kConsumers) {
       // ---- producer: launch r reads a0 (r == 0), buf0 (r odd), buf1 (r even)
       if (lane == 0) {
-        const accel_tmap* map = &a.tmaps[r == 0 ? 0 : ((r & 1u) ? 1 : 2)];
+        const int mi = r == 0 ? 0 : ((r & 1u) ? 1 : 2);
+        const accel_tmap* map = a.gmaps ? a.gmaps + mi : &a.tmaps[mi];
+        if (a.gmaps) tmap_acquire(map);
         // the input was written through the generic proxy (by the previous
         // launch, or -- for a RESOLVE top-up CTA -- by other CTAs of this
         // grid, ordered by the dispatch's wait_complete and the barrier above)

@@ -173,8 +173,8 @@ class MopJob(Job):
 
 class StencilJob(Job):
     TX, TY, TZ = 128, 8, 8
-    # nx % 4 == 0: TMA-staged planes ("stencil_tma", the default) or cp.async
-    # ("stencil"); any nx: "stencil_x"
+    # nx % 4 == 0: cp.async staging ("stencil", the default) or TMA-staged
+    # planes ("stencil_tma"); any nx: "stencil_x"
     KERNELS = ("stencil_tma", "stencil")
 
     def __init__(self, d: dict, device="cuda", kernel: str | None = None):
@@ -187,7 +187,9 @@ class StencilJob(Job):
         self.args = abi.accel_stencil_args(self.inputs["a0"].data_ptr(), self.buf[0].data_ptr(),
                                            self.buf[1].data_ptr(), self.nx, self.ny, self.nz, d["c0"], d["c1"])
         grid = (_cdiv(self.nx, self.TX), _cdiv(self.ny, self.TY), _cdiv(self.nz, self.TZ))
-        kernel = kernel or d.get("kernel") or ("stencil_tma" if self.nx % 4 == 0 else "stencil_x")
+        # default: cp.async staging; stencil_tma is opt-in until its drift next to
+        # bfs is understood (DESIGN.md §6 "stencil staging", scripts/diag_tma.py)
+        kernel = kernel or d.get("kernel") or ("stencil" if self.nx % 4 == 0 else "stencil_x")
         if kernel != "stencil_x" and self.nx % 4:
             raise ValueError(f"{kernel} needs nx % 4 == 0 (16-B rows); stencil_x takes any nx")
         if kernel == "stencil_tma":
@@ -197,6 +199,9 @@ class StencilJob(Job):
             self.args = abi.accel_stencil_tma_args((C.c_uint8 * 384).from_buffer_copy(maps), self.buf[0].data_ptr(),
                                                    self.buf[1].data_ptr(), self.nx, self.ny, self.nz,
                                                    d["c0"], d["c1"])
+            if d.get("tma_global_maps"):   # diagnostic (scripts/diag_tma.py)
+                self.gmaps = torch.frombuffer(bytearray(maps), dtype=torch.uint8).to(self.device)
+                self.args.gmaps = self.gmaps.data_ptr()
         self.kernel = kernel
         self.steps = [Step(kernel, grid, self.args, self.sweeps)]
 

@@ -86,14 +86,14 @@ def test_mop_small_fullcaps(acc, oracle_lib):
                                        ("tiny", dict(nx=129, ny=8, nz=9, sweeps=2)),    # one column past a tile
                                        ("tiny", dict(nx=2, ny=5, nz=4, sweeps=2)),      # all faces
                                        ("small", dict(sweeps=10))])
-@pytest.mark.parametrize("kernel", ["default", "stencil"])
+@pytest.mark.parametrize("kernel", ["default", "stencil_tma"])
 def test_stencil(acc_tiny_caps, oracle_lib, size, over, kernel):
-    """default = stencil_tma (TMA ring) when nx % 4 == 0, stencil_x otherwise;
-    "stencil" = the cp.async staging (nx % 4 == 0 only)."""
+    """default = the cp.async staging ("stencil") when nx % 4 == 0, stencil_x
+    otherwise; "stencil_tma" = the TMA ring (nx % 4 == 0 only)."""
     from paper_conf_cgo_margiolaso16_b200.jobs import StencilJob
     d = synth.preset("stencil", size, **over)
-    if kernel == "stencil" and d["nx"] % 4:
-        pytest.skip("cp.async staging needs nx % 4 == 0")
+    if kernel == "stencil_tma" and d["nx"] % 4:
+        pytest.skip("TMA staging needs nx % 4 == 0")
     k = None if kernel == "default" else kernel
     nat, sh, _ = run_modes(acc_tiny_caps, lambda: StencilJob(d, kernel=k))
     same(nat, sh)
