@@ -57,11 +57,14 @@ struct Kernel {
 };
 
 // A cost-model dequeue order computed on the device (accel_lpt_order<T>) for
-// one (kernel, grid, args); `ready` once its kernel was enqueued (ev recorded).
+// one (kernel, grid, args).  Computed synchronously on the context's order
+// stream the first time a submit needs it -- before anything of the group is
+// enqueued, so a group's first launches still reach the device together (an
+// order kernel on the tenant stream delayed that request's grid and the block
+// scheduler then placed it into whatever room the others left, measured:
+// cutcp 7 CTAs on one SM where the solver's model F had 3).
 struct OrderEntry {
   uint32_t* dev = nullptr;
-  cudaEvent_t ev = nullptr;
-  bool ready = false;
 };
 
 struct Step {
@@ -74,7 +77,6 @@ struct Step {
   uint32_t first;       // first descriptor (relative to the request's slot)
   uint64_t cov_offset;  // coverage offset of the first launch
   const uint32_t* order = nullptr;  // dequeue order (device), nullptr = linear
-  OrderEntry* order_entry = nullptr;  // library-computed order (cache entry)
 };
 
 struct Request {
@@ -187,6 +189,7 @@ struct accel_ctx {
   }
   uint32_t topup_rr = 0;
   cudaStream_t ctl = nullptr;
+  cudaStream_t ostream = nullptr;   // cost-model orders (synchronous, first use)
   cudaEvent_t epoch = nullptr;
   bool epoch_set = false;
   unsigned char* pool = nullptr;
@@ -324,22 +327,6 @@ int enqueue_begin(accel_ctx* ctx, Request* r) {
   CK(ctx, cudaEventRecord(r->ev_arrival, s));
   for (const accel_clear& c : r->clears) CK(ctx, cudaMemsetAsync(c.dst_device, c.value, c.bytes, s));
   for (const accel_copy& c : r->h2d) CK(ctx, cudaMemcpyAsync(c.dst, c.src, c.bytes, cudaMemcpyHostToDevice, s));
-  for (const Step& st : r->steps) {
-    OrderEntry* oe = st.order_entry;
-    if (oe == nullptr) continue;
-    if (!oe->ready) {   // first use: sort the VGs by the kernel's cost model on this stream
-      const Kernel& k = ctx->kernels[st.kid];
-      uint32_t gx = st.grid.x, gy = st.grid.y, gz = st.grid.z;
-      uint32_t* dst = oe->dev;
-      void* params[5] = {const_cast<unsigned char*>(st.args.data()), &gx, &gy, &gz, &dst};
-      CK(ctx, cudaLaunchKernel(k.ofn, dim3(1), dim3(accel::kOrderThreads), params,
-                               accel::kMaxOrderVGs * sizeof(unsigned long long), s));
-      CK(ctx, cudaEventRecord(oe->ev, s));
-      oe->ready = true;
-    } else {
-      CK(ctx, cudaStreamWaitEvent(s, oe->ev, 0));   // computed on another stream
-    }
-  }
   if (r->cov) CK(ctx, cudaMemsetAsync(r->cov, 0, r->cov_elems * sizeof(uint32_t), s));
   if (r->trace) CK(ctx, cudaMemsetAsync(r->trace, 0, r->trace_elems * sizeof(accel_vg_record), s));
   InitParams p{};
@@ -557,12 +544,16 @@ int build_request(accel_ctx* ctx, const accel_request& in, std::unique_ptr<Reque
       key.append(reinterpret_cast<const char*>(&L.grid), sizeof(L.grid));
       key.append(s.args.begin(), s.args.end());
       OrderEntry& oe = ctx->orders[key];
-      if (oe.dev == nullptr) {
+      if (oe.dev == nullptr) {   // first use: sort the VGs by the kernel's cost model now
         CK(ctx, cudaMalloc(&oe.dev, total * sizeof(uint32_t)));
-        CK(ctx, cudaEventCreateWithFlags(&oe.ev, cudaEventDisableTiming));
+        uint32_t gx = L.grid.x, gy = L.grid.y, gz = L.grid.z;
+        uint32_t* dst = oe.dev;
+        void* params[5] = {const_cast<void*>(L.args), &gx, &gy, &gz, &dst};
+        CK(ctx, cudaLaunchKernel(k.ofn, dim3(1), dim3(accel::kOrderThreads), params,
+                                 accel::kMaxOrderVGs * sizeof(unsigned long long), ctx->ostream));
+        CK(ctx, cudaStreamSynchronize(ctx->ostream));
       }
       s.order = oe.dev;
-      s.order_entry = &oe;
     }
     s.quota = s.total;
     s.first = n_desc;
@@ -833,6 +824,8 @@ int accel_init(const accel_config* cfg, accel_ctx** out) {
       return init_fail(e, "cudaStreamCreate");
   if ((e = cudaStreamCreateWithFlags(&ctx->ctl, cudaStreamNonBlocking)) != cudaSuccess)
     return init_fail(e, "cudaStreamCreate");
+  if ((e = cudaStreamCreateWithFlags(&ctx->ostream, cudaStreamNonBlocking)) != cudaSuccess)
+    return init_fail(e, "cudaStreamCreate");
   if ((e = cudaEventCreate(&ctx->epoch)) != cudaSuccess) return init_fail(e, "cudaEventCreate");
   if ((e = cudaMalloc(&ctx->pool, (size_t)kPoolSlots * kDescBytes)) != cudaSuccess)
     return init_fail(e, "cudaMalloc(pool)");
@@ -861,10 +854,8 @@ int accel_finalize(accel_ctx* ctx) {
     release_request(ctx, kv.second.get());
   }
   ctx->reqs.clear();
-  for (auto& kv : ctx->orders) {
+  for (auto& kv : ctx->orders)
     if (kv.second.dev) cudaFree(kv.second.dev);
-    if (kv.second.ev) cudaEventDestroy(kv.second.ev);
-  }
   ctx->orders.clear();
   for (cudaEvent_t ev : ctx->free_events) cudaEventDestroy(ev);
   for (int t = 0; t < ACCEL_MAX_TENANTS; ++t)
@@ -872,6 +863,7 @@ int accel_finalize(accel_ctx* ctx) {
   for (int t = 0; t < accel_ctx::kTopupStreams; ++t)
     if (ctx->topup[t]) cudaStreamDestroy(ctx->topup[t]);
   if (ctx->ctl) cudaStreamDestroy(ctx->ctl);
+  if (ctx->ostream) cudaStreamDestroy(ctx->ostream);
   if (ctx->epoch) cudaEventDestroy(ctx->epoch);
   if (ctx->pool) cudaFree(ctx->pool);
   if (ctx->ctl_pool) cudaFree(ctx->ctl_pool);
@@ -1208,8 +1200,8 @@ int accel_dequeue_order(accel_ctx* ctx, int32_t kernel_id, const accel_dim3* gri
   uint32_t gx = grid->x, gy = grid->y, gz = grid->z;
   void* params[5] = {const_cast<void*>(args), &gx, &gy, &gz, &order_device};
   CK(ctx, cudaLaunchKernel(k.ofn, dim3(1), dim3(accel::kOrderThreads), params,
-                           accel::kMaxOrderVGs * sizeof(unsigned long long), ctx->ctl));
-  CK(ctx, cudaStreamSynchronize(ctx->ctl));
+                           accel::kMaxOrderVGs * sizeof(unsigned long long), ctx->ostream));
+  CK(ctx, cudaStreamSynchronize(ctx->ostream));
   return ACCEL_OK;
 }
 

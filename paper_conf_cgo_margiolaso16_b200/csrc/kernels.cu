@@ -110,6 +110,7 @@ const Builtin kBuiltins[] = {
     {"mop", &make_desc<Mop>},
     {"stencil", &make_desc<Stencil>},
     {"stencil_x", &make_desc<StencilX>},
+    {"stencil_deep", &make_desc<StencilDeep>},
     {"stencil_tma", &make_desc<StencilTma>},
     {"histo", &make_desc<Histo>},
     {"histo_wide", &make_desc<HistoWide>},

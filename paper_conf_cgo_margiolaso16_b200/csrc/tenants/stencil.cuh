@@ -31,21 +31,24 @@ namespace accel {
 // cp.async copies, each column checked against nx, outputs stored per
 // element.  Two kernels rather than a branch: the ragged path's registers
 // would otherwise count against the aligned one (it spilled).
-template <bool kAligned>
+#ifndef STENCIL_KD
+#define STENCIL_KD 4
+#endif
+// kDepth: planes in flight beyond z+1 ("stencil_deep": the whole 10-plane
+// tile in flight per VG -- more bytes in flight per CTA for a small share)
+template <bool kAligned, int kDepth = STENCIL_KD>
 struct StencilT {
   using Args = accel_stencil_args;
   static constexpr int kThreads = 256;
   static constexpr int kTX = 128, kTY = 8, kTZ = 8;
   static constexpr uint32_t kChunk = 1;
-  static constexpr int kMinBlocks = kAligned ? 5 : 4;   // the ragged path needs a few more registers
+  // the ragged path needs a few more registers; the deep ring (55 KB) fits 4 per SM
+  static constexpr int kMinBlocks = (kAligned && kDepth <= 4) ? 5 : 4;
   static constexpr int kRows = kTY + 2;                 // y halo
   static constexpr int kCols = kTX + 8;                 // x0-4 .. x0+131 (16-B multiples)
   static constexpr uint32_t kPlaneBytes = kRows * kCols * 4;          // 5440
   static constexpr uint32_t kSlot = (kPlaneBytes + 127) / 128 * 128;  // 5504
-#ifndef STENCIL_KD
-#define STENCIL_KD 4
-#endif
-  static constexpr int kD = STENCIL_KD;                 // planes in flight beyond z+1
+  static constexpr int kD = kDepth;                     // planes in flight beyond z+1
   static constexpr int kR = kD + 2;                     // ring slots
 #ifndef STENCIL_MBAR
 #define STENCIL_MBAR 0
@@ -265,5 +268,6 @@ struct StencilT {
 
 using Stencil = StencilT<true>;
 using StencilX = StencilT<false>;
+using StencilDeep = StencilT<true, 8>;
 
 }  // namespace accel

@@ -12,6 +12,7 @@ sequence as one request (DESIGN.md R-job-1).
 from __future__ import annotations
 
 import ctypes as C
+import os
 from dataclasses import dataclass, field
 
 import numpy as np
@@ -189,7 +190,8 @@ class StencilJob(Job):
         grid = (_cdiv(self.nx, self.TX), _cdiv(self.ny, self.TY), _cdiv(self.nz, self.TZ))
         # default: cp.async staging; stencil_tma is opt-in until its drift next to
         # bfs is understood (DESIGN.md §6 "stencil staging", scripts/diag_tma.py)
-        kernel = kernel or d.get("kernel") or ("stencil" if self.nx % 4 == 0 else "stencil_x")
+        kernel = kernel or d.get("kernel") or os.environ.get("ACCEL_STENCIL_KERNEL") or \
+            ("stencil" if self.nx % 4 == 0 else "stencil_x")
         if kernel != "stencil_x" and self.nx % 4:
             raise ValueError(f"{kernel} needs nx % 4 == 0 (16-B rows); stencil_x takes any nx")
         if kernel == "stencil_tma":
