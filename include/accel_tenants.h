@@ -116,15 +116,18 @@ typedef struct {
 } accel_cutcp_args;
 
 /* tpacf -- angular two-point correlation histograms, SoA unit vectors.
- * block 256, VG = (set s in [0, 2*nsets], 256-point block i): s == 0 -> DD,
- * s = 1..nsets -> RR of set s-1, s = nsets+1..2*nsets -> DR of set
- * s-nsets-1; grid (ceil(npts/256), 2*nsets+1).  dd/rr/dr u64[nedges+1],
- * cleared by the request. */
+ * block 256, VG = (256-point block i, set s in [0, 2*nsets], part q): s == 0
+ * -> DD, s = 1..nsets -> RR of set s-1, s = nsets+1..2*nsets -> DR of set
+ * s-nsets-1; the VG pairs its points with part q of the 256-point tiles of
+ * the other set (the tiles split into qsplit near-equal runs; DD/RR tiles
+ * start at the diagonal one); grid (ceil(npts/256), 2*nsets+1, qsplit).
+ * dd/rr/dr u64[nedges+1], cleared by the request. */
 typedef struct {
   const float *data;   /* [3][npts]          */
   const float *rand;   /* [nsets][3][npts]   */
   const float *binb;   /* [nedges] descending */
   uint32_t npts, nsets, nedges;
+  uint32_t qsplit;     /* >= 1 */
   unsigned long long *dd, *rr, *dr;
 } accel_tpacf_args;
 

@@ -136,7 +136,7 @@ class accel_cutcp_args(C.Structure):
 
 class accel_tpacf_args(C.Structure):
     _fields_ = [("data", vp), ("rand", vp), ("binb", vp), ("npts", u32), ("nsets", u32),
-                ("nedges", u32), ("dd", vp), ("rr", vp), ("dr", vp)]
+                ("nedges", u32), ("qsplit", u32), ("dd", vp), ("rr", vp), ("dr", vp)]
 
 
 class accel_spmv_args(C.Structure):

@@ -8,14 +8,18 @@
 // angular bin of a pair is decided on the fp32 dot product
 // (x*x' + y*y') + z*z' (round-to-nearest, no FMA, DESIGN.md R-fp-1) by a
 // binary search over the descending bin edges; each lane counts into its own
-// shared-memory sub-histogram column (conflict-free, no atomics); the VG ends
-// with one 64-bit global atomic per bin.  Integer result: bit-exact.
+// shared-memory sub-histogram column (bank = lane, conflict-free) with one
+// shared-memory RED.ADD per pair (TPACF_REDS=0: load + add + store); the VG
+// ends with one 64-bit global atomic per bin.  Integer result: bit-exact.
 #pragma once
 #include "../device/dispatch.cuh"
 #include "accel_tenants.h"
 
 #ifndef TPACF_REDS
 #define TPACF_REDS 1
+#endif
+#ifndef TPACF_UNROLL2
+#define TPACF_UNROLL2 1
 #endif
 
 namespace accel {
@@ -37,8 +41,22 @@ struct Tpacf {
   // Dequeue-order cost model (dispatch.cuh accel_lpt_order): Q tiles the VG
   // walks -- DD / RR blocks (y <= S) start at their diagonal tile, DR blocks
   // (y > S) walk all of them.
+  // Q tiles [t0, t1) of VG vb: part vb.z of the run that starts at the
+  // diagonal tile (DD / RR: pairs i < j) or at tile 0 (DR)
+  static __device__ __forceinline__ void tile_range(const Args& a, const VirtualBlock& vb, uint32_t& t0,
+                                                    uint32_t& t1) {
+    const uint32_t ntiles = (a.npts + kTile - 1) / kTile;
+    const uint32_t first = vb.y <= a.nsets ? vb.x : 0u;
+    const uint32_t len = ntiles - first, parts = vb.gz;
+    t0 = first + (uint32_t)(((uint64_t)len * vb.z) / parts);
+    t1 = first + (uint32_t)(((uint64_t)len * (vb.z + 1)) / parts);
+  }
+
   static __device__ float vg_cost(const Args& a, const VirtualBlock& vb) {
-    return vb.y <= a.nsets ? (float)vb.gx - (float)vb.x - 0.5f : (float)vb.gx;
+    uint32_t t0, t1;
+    tile_range(a, vb, t0, t1);
+    // the diagonal tile holds half its pairs
+    return (float)(t1 - t0) - ((vb.y <= a.nsets && t0 == vb.x && t1 > t0) ? 0.5f : 0.f);
   }
 
   static __device__ __forceinline__ void body(const Args& a, const VirtualBlock& vb, char* smem) {
@@ -75,8 +93,9 @@ struct Tpacf {
     uint32_t* myh = hist + warp * kMaxBins * 32 + lane;
     __syncthreads();   // edges staged
     const float e7 = edges[7], e15 = edges[15], e23 = edges[23];
-    const uint32_t j_first_tile = upper ? vb.x * kTile : 0;
-    for (uint32_t jt = j_first_tile; jt < n; jt += kTile) {
+    uint32_t tile0, tile1;
+    tile_range(a, vb, tile0, tile1);
+    for (uint32_t jt = tile0 * kTile; jt < tile1 * kTile; jt += kTile) {
       __syncthreads();
       const uint32_t jj = jt + t;
       if (jj < n) qt[t] = make_float4(__ldg(Q + jj), __ldg(Q + n + jj), __ldg(Q + 2 * n + jj), 0.f);
@@ -85,16 +104,20 @@ struct Tpacf {
       const uint32_t cnt = min((uint32_t)kTile, n - jt);
       // pairs i < j on the diagonal tile start after i
       const uint32_t q0 = (upper && jt == vb.x * kTile) ? (uint32_t)t + 1 : 0u;
-      for (uint32_t q = q0; q < cnt; ++q) {
-        const float4 qv = qt[q];
-        const float d = __fadd_rn(__fadd_rn(__fmul_rn(ix, qv.x), __fmul_rn(iy, qv.y)), __fmul_rn(iz, qv.z));
-        // bin = #{k : d < edges[k]}; edges descending -> binary search, its
-        // first two levels from registers (edges[15], then edges[7] / [23])
+      // bin = #{k : d < edges[k]}; edges descending -> binary search, its
+      // first two levels from registers (edges[15], then edges[7] / [23])
+      auto bin_of = [&](float d) {
         int m = (e15 > d) ? 16 : 0;
         if (((m != 0) ? e23 : e7) > d) m += 8;
 #pragma unroll
         for (int step = 4; step >= 1; step >>= 1)
           if (edges[m + step - 1] > d) m += step;
+        return m;
+      };
+      auto dot = [&](const float4& qv) {
+        return __fadd_rn(__fadd_rn(__fmul_rn(ix, qv.x), __fmul_rn(iy, qv.y)), __fmul_rn(iz, qv.z));
+      };
+      auto count = [&](int m) {
 #if TPACF_REDS
         // lane-private counter (bank = lane): one RED.ADD on shared memory
         // instead of load + add + store
@@ -102,7 +125,18 @@ struct Tpacf {
 #else
         myh[m * 32] += 1u;
 #endif
+      };
+      uint32_t q = q0;
+#if TPACF_UNROLL2
+      // two independent search chains in flight (their shared-memory edge
+      // loads overlap)
+      for (; q + 1 < cnt; q += 2) {
+        const int m0 = bin_of(dot(qt[q])), m1 = bin_of(dot(qt[q + 1]));
+        count(m0);
+        count(m1);
       }
+#endif
+      for (; q < cnt; ++q) count(bin_of(dot(qt[q])));
     }
     __syncthreads();
     if (t < (int)ne + 1) {

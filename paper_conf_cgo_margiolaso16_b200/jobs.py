@@ -224,7 +224,10 @@ class HistoJob(Job):
             raise ValueError("histo: 1..16384 bins; u8 samples need 256 bins")
         # > 4096 bins: the packed 16-bit private histogram (VGs < 65536 samples)
         self.kernel = "histo" if self.bins <= 4096 else "histo_wide"
-        self.per_vg = 4096 if self.sb == 1 else d.get("per_vg", 16384)
+        # samples per VG: histo_wide flushes up to 16K bins per VG with global
+        # atomics, so its VGs are as large as the 16-bit counters allow
+        # (measured at the SURVEY default: 74 -> 52 us per pass, 16384 -> 61440)
+        self.per_vg = 4096 if self.sb == 1 else d.get("per_vg", 16384 if self.kernel == "histo" else 61440)
         assert self.per_vg % 4096 == 0 and (self.kernel == "histo" or self.per_vg < 65536)
         self.inputs = {"samples": _dev(d["samples"], self.device)}
         self.hist = torch.zeros(2 * self.bins, dtype=torch.int32, device=self.device)
@@ -339,11 +342,13 @@ class TpacfJob(Job):
         self.hists = torch.zeros(3 * nb, dtype=torch.int64, device=self.device)
         self.out = {"hists": self.hists}
         p = self.hists.data_ptr()
+        # VGs split the other set's tiles in `qsplit` runs: finer VGs, shorter tail
+        self.qsplit = int(d.get("qsplit", os.environ.get("ACCEL_TPACF_QSPLIT", 2)))
         self.args = abi.accel_tpacf_args(self.inputs["data"].data_ptr(), self.inputs["rand"].data_ptr(),
-                                         self.inputs["binb"].data_ptr(), self.n, self.S, self.nedges,
+                                         self.inputs["binb"].data_ptr(), self.n, self.S, self.nedges, self.qsplit,
                                          p, p + 8 * nb, p + 16 * nb)
         self.clears = [(self.hists, 0)]
-        grid = (_cdiv(self.n, 256), 2 * self.S + 1, 1)
+        grid = (_cdiv(self.n, 256), 2 * self.S + 1, self.qsplit)
         # dequeue order: the library's cost model (Tpacf::vg_cost, longest pair blocks first)
         self.steps = [Step("tpacf", grid, self.args, 1)]
 

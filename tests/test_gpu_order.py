@@ -50,11 +50,19 @@ def cutcp_cost(d, grid):
     return cost
 
 
-def tpacf_cost(S, grid):
-    gx, gy, _ = grid
-    x = np.tile(np.arange(gx), gy)
-    y = np.repeat(np.arange(gy), gx)
-    return np.where(y <= S, gx - x - 0.5, gx).astype(np.float64)
+def tpacf_cost(S, n, grid):
+    """Q tiles per VG (x, y, part z): part z of the tiles from the diagonal
+    one (DD/RR, y <= S) or from tile 0 (DR), the diagonal tile half-counted."""
+    gx, gy, gz = grid
+    ntiles = -(-n // 256)
+    cost = np.zeros(gx * gy * gz)
+    for v in range(gx * gy * gz):
+        x, y, z = v % gx, (v // gx) % gy, v // (gx * gy)
+        first = x if y <= S else 0
+        ln = ntiles - first
+        t0, t1 = first + ln * z // gz, first + ln * (z + 1) // gz
+        cost[v] = (t1 - t0) - (0.5 if (y <= S and t0 == x and t1 > t0) else 0.0)
+    return cost
 
 
 @pytest.mark.parametrize("tenant,size", [("cutcp", "tiny"), ("cutcp", "small"), ("tpacf", "tiny"),
@@ -76,7 +84,7 @@ def test_library_order_is_lpt_of_the_cost_model(tenant, size):
         abi.accel_dequeue_order(acc.ctx, acc.kids[st.kernel], st.grid, st.args, out.data_ptr())
         got = out.cpu().numpy().astype(np.int64)
     assert np.array_equal(np.sort(got), np.arange(g))             # a permutation
-    cost = cutcp_cost(d, st.grid) if tenant == "cutcp" else tpacf_cost(d["nsets"], st.grid)
+    cost = cutcp_cost(d, st.grid) if tenant == "cutcp" else tpacf_cost(d["nsets"], d["npts"], st.grid)
     # non-increasing cost along the order, ties by increasing id
     c = cost[got]
     assert (np.diff(c) <= 0).all()

@@ -335,3 +335,15 @@ def test_stencil_bit_exact_fp32_sequence(acc_tiny_caps, kernel, over):
     nat, sh, _ = run_modes(acc_tiny_caps, lambda: StencilJob(d, kernel=kernel))
     ref = _stencil_fp32_replica(d)
     assert np.array_equal(nat["a"], ref) and np.array_equal(sh["a"], ref)
+
+
+@pytest.mark.parametrize("qsplit", [1, 3, 7])
+def test_tpacf_qsplit(acc_tiny_caps, oracle_lib, qsplit):
+    """VGs over parts of the other set's tiles (any split, including more
+    parts than a DD/RR block has tiles) count every pair exactly once."""
+    from paper_conf_cgo_margiolaso16_b200.jobs import TpacfJob
+    d = dict(synth.preset("tpacf", "small", seed=8), qsplit=qsplit)
+    nat, sh, _ = run_modes(acc_tiny_caps, lambda: TpacfJob(d))
+    dd, rr, dr = oracle_lib.tpacf(d)
+    for r in (nat, sh):
+        assert np.array_equal(r["dd"], dd) and np.array_equal(r["rr"], rr) and np.array_equal(r["dr"], dr)
