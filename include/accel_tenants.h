@@ -184,6 +184,26 @@ typedef struct {
   uint32_t m, n, k;
 } accel_sgemm_tc_args;
 
+/* sad -- Parboil "sad" (H.264 motion estimation), three
+ * kernels sharing one argument struct, run as the three steps of a request:
+ *   "sad_4x4"   sad4[mb][p][b] = sum over the 4x4 sub-block b of the 16x16
+ *               macroblock mb of |cur - ref displaced by (dx, dy)|, every
+ *               (dx, dy) in [-R, R]^2 (p = (dy+R)(2R+1) + dx+R), reference
+ *               coordinates clamped to the frame; VG = macroblock, grid
+ *               (w/16, h/16), block 256, R <= 16
+ *   "sad_8x8"   sad8[mb][p][q]: the four 8x8 sums of sad4; same grid
+ *   "sad_16x16" sad16[mb][p]: the 16x16 sum of sad8; same grid
+ * w, h multiples of 16; u16 pixels < 256 (so every SAD fits u16); DEVICE
+ * buffers: cur/ref [h][w], sad4 [mbs][(2R+1)^2][16], sad8 [..][4], sad16 [..]. */
+typedef struct {
+  const uint16_t *cur;
+  const uint16_t *ref;
+  uint16_t *sad4;
+  uint16_t *sad8;
+  uint16_t *sad16;
+  uint32_t w, h, R;
+} accel_sad_args;
+
 /* mri-q ComputePhiMag: phimag = phir^2 + phii^2.  block 256, grid ceil(numk/256). */
 typedef struct {
   const float *phir;

@@ -142,3 +142,14 @@ def mriq(d: dict):
     pm = mriq_phimag(d)
     qr, qi = mriq_points(d, np.arange(d["numx"]), pm)
     return pm, qr, qi
+
+
+def sad(d: dict):
+    """(sad4 u16[mb][p][16], sad8 u16[mb][p][4], sad16 u16[mb][p])."""
+    nmb = (d["w"] // 16) * (d["h"] // 16)
+    npos = (2 * d["R"] + 1) ** 2
+    s4 = np.empty((nmb, npos, 16), dtype=np.uint16)
+    s8 = np.empty((nmb, npos, 4), dtype=np.uint16)
+    s16 = np.empty((nmb, npos), dtype=np.uint16)
+    lib().oracle_sad(_p(d["cur"]), _p(d["ref"]), I64(d["w"]), I64(d["h"]), I64(d["R"]), _p(s4), _p(s8), _p(s16))
+    return s4, s8, s16

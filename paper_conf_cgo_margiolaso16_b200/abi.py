@@ -162,6 +162,13 @@ accel_stencil_deep_args = accel_stencil_args
 accel_histo_wide_args = accel_histo_args
 
 
+class accel_sad_args(C.Structure):
+    _fields_ = [("cur", vp), ("ref", vp), ("sad4", vp), ("sad8", vp), ("sad16", vp), ("w", u32), ("h", u32), ("R", u32)]
+
+
+accel_sad_4x4_args = accel_sad_8x8_args = accel_sad_16x16_args = accel_sad_args
+
+
 class accel_mriq_phimag_args(C.Structure):
     _fields_ = [("phir", vp), ("phii", vp), ("phimag", vp), ("numk", u32)]
 

@@ -12,6 +12,7 @@
 #include "tenants/histo.cuh"
 #include "tenants/mop.cuh"
 #include "tenants/mriq.cuh"
+#include "tenants/sad.cuh"
 #include "tenants/sgemm.cuh"
 #include "tenants/sgemm_tc.cuh"
 #include "tenants/spmv.cuh"
@@ -121,6 +122,9 @@ const Builtin kBuiltins[] = {
     {"sgemm", &make_desc<Sgemm>},
     {"sgemm_split", &make_desc<SgemmSplit>},
     {"sgemm_tc", &make_desc<SgemmTc>},
+    {"sad_4x4", &make_desc<Sad4>},
+    {"sad_8x8", &make_desc<Sad8>},
+    {"sad_16x16", &make_desc<Sad16>},
     {"mriq_phimag", &make_desc<MriqPhiMag>},
     {"mriq_q", &make_desc<MriqQ>},
 };

@@ -474,8 +474,45 @@ class MriqJob(Job):
                 "skip_launches": 1, "flops_per_launch": 11.0 * pairs, "peak_tflops": FP32_SIMT_TFLOPS}
 
 
+class SadJob(Job):
+    """Parboil sad (f3): three steps -- 4x4 SADs over the search window, then
+    the 8x8 and 16x16 sums -- one request (R-solver-8; main step = 4x4)."""
+
+    def __init__(self, d: dict, device="cuda"):
+        super().__init__(name="sad", device=torch.device(device))
+        self.w, self.h, self.R = d["w"], d["h"], d["R"]
+        if self.w % 16 or self.h % 16 or not 0 <= self.R <= 16:
+            raise ValueError("sad: w, h multiples of 16 and R <= 16")
+        self.inputs = {"cur": _dev(d["cur"].view(np.int16), self.device),
+                       "ref": _dev(d["ref"].view(np.int16), self.device)}
+        nmb, npos = (self.w // 16) * (self.h // 16), (2 * self.R + 1) ** 2
+        self.nmb, self.npos = nmb, npos
+        self.s4 = torch.empty(nmb * npos * 16, dtype=torch.int16, device=self.device)
+        self.s8 = torch.empty(nmb * npos * 4, dtype=torch.int16, device=self.device)
+        self.s16 = torch.empty(nmb * npos, dtype=torch.int16, device=self.device)
+        self.out = {"sad4": self.s4, "sad8": self.s8, "sad16": self.s16}
+        self.args = abi.accel_sad_args(self.inputs["cur"].data_ptr(), self.inputs["ref"].data_ptr(),
+                                       self.s4.data_ptr(), self.s8.data_ptr(), self.s16.data_ptr(),
+                                       self.w, self.h, self.R)
+        grid = (self.w // 16, self.h // 16, 1)
+        self.main_step = 0
+        self.steps = [Step("sad_4x4", grid, self.args, 1), Step("sad_8x8", grid, self.args, 1),
+                      Step("sad_16x16", grid, self.args, 1)]
+
+    def result(self):
+        return {"sad4": _np(self.s4, np.uint16).reshape(self.nmb, self.npos, 16),
+                "sad8": _np(self.s8, np.uint16).reshape(self.nmb, self.npos, 4),
+                "sad16": _np(self.s16, np.uint16).reshape(self.nmb, self.npos)}
+
+    def work(self):
+        # the dominant (4x4) launch: 256 absolute differences per (macroblock, displacement)
+        n = self.nmb * self.npos
+        return {"ops": 256 * n, "bytes": 2 * 16 * n + 4 * self.w * self.h, "bound": "alu", "launches": 3,
+                "skip_launches": 0, "flops_per_launch": 2.0 * 256 * n, "peak_tflops": FP32_SIMT_TFLOPS}
+
+
 JOBS = {"mop": MopJob, "stencil": StencilJob, "histo": HistoJob, "bfs": BfsJob, "cutcp": CutcpJob,
-        "tpacf": TpacfJob, "spmv": SpmvJob, "sgemm": SgemmTcJob, "sgemm_simt": SgemmJob, "mriq": MriqJob}
+        "tpacf": TpacfJob, "spmv": SpmvJob, "sgemm": SgemmTcJob, "sgemm_simt": SgemmJob, "mriq": MriqJob, "sad": SadJob}
 
 
 def make_job(name: str, d: dict, device="cuda") -> Job:

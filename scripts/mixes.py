@@ -41,6 +41,7 @@ from paper_conf_cgo_margiolaso16_b200.jobs import make_job  # noqa: E402
 from paper_conf_cgo_margiolaso16_b200.runtime import Accel  # noqa: E402
 
 TENANTS = ["bfs", "cutcp", "stencil", "tpacf", "histo", "spmv", "sgemm", "mriq"]
+ALPHA = 0.0   # --alpha: SHARED-mode weights ~ T(a)^alpha (0 = equal shares, the paper's policy)
 MODES = [("native", abi.MODE_NATIVE, abi.POLICY_STATIC), ("resolve", abi.MODE_SHARED, abi.POLICY_RESOLVE),
          ("static", abi.MODE_SHARED, abi.POLICY_STATIC)]
 SHARED = ["resolve", "static"]
@@ -69,15 +70,16 @@ class Runner:
         if self.acc.mode != mode or self.acc.policy != policy:
             self.acc.set_mode(mode, policy)
 
-    def run(self, jobs, mode, policy, delays_s=None):
-        """Submit `jobs` (arrival order); delays_s[i] = host-side arrival offset."""
+    def run(self, jobs, mode, policy, delays_s=None, weights=None):
+        """Submit `jobs` (arrival order); delays_s[i] = host-side arrival offset;
+        weights = sharing ratios, None = equal."""
         self.set(mode, policy)
         self.flush_buf.fill_(1.0)
         torch.cuda.synchronize()
         self.acc.epoch()
         ids = []
         if delays_s is None:
-            ids = self.acc.submit(jobs, tenants=list(range(len(jobs))))
+            ids = self.acc.submit(jobs, tenants=list(range(len(jobs))), weights=weights)
         else:
             t0 = time.perf_counter()
             for i, (j, dl) in enumerate(zip(jobs, delays_s)):
@@ -187,7 +189,13 @@ def sampled(r: Runner, ta, reps, k, n, seed, repeat=False):
             seen[t] = seen.get(t, 0) + 1
         res = {"mix": names}
         for name, mode, pol in MODES:
-            runs = [mix_metrics(r.run(jobs, mode, pol), [ta[t] for t in names]) for _ in range(reps)]
+            w = None
+            if ALPHA and mode == abi.MODE_SHARED:
+                # profile-guided sharing ratio: w ~ T(a)^alpha (alpha < 0: the
+                # shorter requests get the larger shares)
+                tmax = max(ta[t] for t in names)
+                w = [max(1, round(16 * (ta[t] / tmax) ** ALPHA)) for t in names]
+            runs = [mix_metrics(r.run(jobs, mode, pol, weights=w), [ta[t] for t in names]) for _ in range(reps)]
             res[name] = {kk: statistics.mean(x[kk] for x in runs) for kk in keys}
         mixes.append(res)
         print(json.dumps({"mix": names, **{nm: {kk: round(v, 3) for kk, v in res[nm].items()} for nm, _, _ in MODES}}),
@@ -223,6 +231,7 @@ def main():
     ap.add_argument("--n", type=int, default=32, help="f2: number of sampled mixes")
     ap.add_argument("--seed", type=int, default=2024)
     ap.add_argument("--repeat", action="store_true", help="f2: tuples with repetition (the paper's space)")
+    ap.add_argument("--alpha", type=float, default=0.0, help="f2: SHARED weights ~ T(a)^alpha (0 = equal)")
     ap.add_argument("--reps", type=int, default=3)
     ap.add_argument("--size", default="default")
     ap.add_argument("--out", default=None)
@@ -230,6 +239,8 @@ def main():
     ap.add_argument("--tenants", default=None, help="restrict the tenants loaded (comma-separated)")
     ap.add_argument("--modes", default=None, help="restrict the modes (comma-separated; native is always run)")
     a = ap.parse_args()
+    global ALPHA
+    ALPHA = a.alpha
     dev = torch.device("cuda", 0)
     if a.tenants:
         TENANTS[:] = a.tenants.split(",")

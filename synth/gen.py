@@ -20,6 +20,7 @@ __all__ = [
     "gen_spmv",
     "gen_sgemm",
     "gen_mriq",
+    "gen_sad",
     "GENERATORS",
 ]
 
@@ -208,8 +209,27 @@ def gen_mriq(nvox_1d: int, numk: int, seed: int = 0) -> dict:
     }
 
 
+def gen_sad(w: int, h: int, R: int = 16, seed: int = 0) -> dict:
+    """Two video frames (u16 pixels < 256): a smooth random field (sum of
+    Gaussian-blurred noise octaves) and the same field moved by a seeded
+    global shift plus noise -- motion-estimation-shaped input [ext Parboil sad]."""
+    r = rng(seed)
+    base = np.zeros((h + 64, w + 64))
+    for sc in (1, 4, 16):
+        nz = r.normal(0.0, 1.0, ((h + 64) // sc + 2, (w + 64) // sc + 2))
+        up = np.kron(nz, np.ones((sc, sc)))[: h + 64, : w + 64]
+        base += up * sc
+    base = (base - base.min()) / (base.max() - base.min()) * 255.0
+    sy, sx = (int(v) for v in r.integers(-6, 7, 2))
+    cur = base[32: 32 + h, 32: 32 + w]
+    ref = base[32 + sy: 32 + sy + h, 32 + sx: 32 + sx + w] + r.normal(0.0, 3.0, (h, w))
+    q = lambda a: np.clip(np.rint(a), 0, 255).astype(np.uint16)  # noqa: E731
+    return {"cur": np.ascontiguousarray(q(cur)), "ref": np.ascontiguousarray(q(ref)),
+            "w": int(w), "h": int(h), "R": int(R)}
+
+
 GENERATORS = {
     "mop": gen_mop, "stencil": gen_stencil, "histo": gen_histo, "bfs": gen_bfs,
     "cutcp": gen_cutcp, "tpacf": gen_tpacf, "spmv": gen_spmv, "sgemm": gen_sgemm,
-    "mriq": gen_mriq,
+    "mriq": gen_mriq, "sad": gen_sad,
 }

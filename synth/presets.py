@@ -55,6 +55,11 @@ PRESETS: dict[str, dict[str, dict]] = {
         "small": dict(m=1024, n=1056, k=992),
         "default": dict(m=4096, n=4096, k=4096),
     },
+    "sad": {
+        "tiny": dict(w=48, h=32, R=4),
+        "small": dict(w=176, h=144, R=16),     # QCIF
+        "default": dict(w=1920, h=1072, R=16),  # [ext Parboil sad large]
+    },
     "mriq": {
         "tiny": dict(nvox_1d=12, numk=300),
         "small": dict(nvox_1d=32, numk=3072),

@@ -87,3 +87,25 @@ def test_mriq_default_sampled(acc, oracle_lib):
     qr, qi = oracle_lib.mriq_points(d, idx, pm)
     assert_close_fp32(np.concatenate([res["qr"][idx], res["qi"][idx]]), np.concatenate([qr, qi]),
                       what="mri-q default")
+
+
+# ---------------------------------------------------------------- sad (f3)
+@pytest.mark.parametrize("size,over", [("tiny", {}), ("small", {}), ("tiny", dict(R=0)), ("tiny", dict(R=7, w=64))])
+def test_sad(acc_tiny_caps, oracle_lib, size, over):
+    """Parboil sad, three steps (4x4 SADs, 8x8 and 16x16 sums): bit-exact in
+    both modes, every displacement parity and the frame-edge clamping."""
+    from paper_conf_cgo_margiolaso16_b200.jobs import SadJob
+    d = synth.preset("sad", size, **over)
+    nat, sh, _ = run_modes(acc_tiny_caps, lambda: SadJob(d))
+    s4, s8, s16 = oracle_lib.sad(d)
+    for r in (nat, sh):
+        assert np.array_equal(r["sad4"], s4) and np.array_equal(r["sad8"], s8) and np.array_equal(r["sad16"], s16)
+
+
+def test_sad_default(acc, oracle_lib):
+    from paper_conf_cgo_margiolaso16_b200.jobs import SadJob
+    d = synth.preset("sad", "default")
+    nat, sh, _ = run_modes(acc, lambda: SadJob(d))
+    s4, s8, s16 = oracle_lib.sad(d)
+    for r in (nat, sh):
+        assert np.array_equal(r["sad16"], s16) and np.array_equal(r["sad8"], s8) and np.array_equal(r["sad4"], s4)

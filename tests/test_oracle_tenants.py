@@ -327,3 +327,60 @@ def test_mriq_origin_and_dc():
               phir=d["phir"][5:6].copy(), phii=d["phii"][5:6].copy())
     qr, qi = T().mriq_points(d1, np.arange(50))
     assert np.all(qr == np.float64(T().mriq_phimag(d1)[0])) and np.all(qi == 0.0)
+
+
+# ---- sad (Parboil "sad") ----------------------------------
+
+def _sad_numpy(d):
+    """numpy brute force of the 4x4 SADs: the reference frame padded by edge
+    replication (= clamping), every displacement sliced out at once."""
+    w, h, R = d["w"], d["h"], d["R"]
+    cur = d["cur"].astype(np.int64)
+    ref = np.pad(d["ref"].astype(np.int64), R, mode="edge")
+    side = 2 * R + 1
+    out = np.empty((h // 16 * (w // 16), side * side, 16), dtype=np.int64)
+    for p in range(side * side):
+        dy, dx = p // side - R, p % side - R
+        diff = np.abs(cur - ref[R + dy: R + dy + h, R + dx: R + dx + w])
+        blk = diff.reshape(h // 4, 4, w // 4, 4).sum(axis=(1, 3))          # [h/4][w/4] 4x4 sums
+        mbs = blk.reshape(h // 16, 4, w // 16, 4).transpose(0, 2, 1, 3)    # [my][mx][by][bx]
+        out[:, p, :] = mbs.reshape(-1, 16)
+    return out
+
+
+def test_sad_matches_numpy_bruteforce():
+    d = synth.preset("sad", "tiny", seed=3)
+    s4, s8, s16 = T().sad(d)
+    ref4 = _sad_numpy(d)
+    assert np.array_equal(s4.astype(np.int64), ref4)
+    # the 8x8 / 16x16 levels are the sums of the 4x4 SADs they cover
+    q = ref4.reshape(ref4.shape[0], ref4.shape[1], 2, 2, 2, 2).sum(axis=(3, 5))   # [by2][bx2]
+    assert np.array_equal(s8.astype(np.int64), q.reshape(ref4.shape[0], ref4.shape[1], 4))
+    assert np.array_equal(s16.astype(np.int64), ref4.sum(axis=2))
+
+
+def test_sad_identical_frames_zero_at_centre():
+    d = synth.preset("sad", "tiny", seed=4)
+    d = dict(d, ref=d["cur"].copy())
+    s4, _, s16 = T().sad(d)
+    centre = d["R"] * (2 * d["R"] + 1) + d["R"]
+    assert not s4[:, centre, :].any() and not s16[:, centre].any()
+    assert (s16[:, np.arange(s16.shape[1]) != centre] > 0).any()
+
+
+def test_sad_global_shift_is_found():
+    """ref = cur moved by (sx, sy) (no noise): every macroblock whose displaced
+    block stays inside the frame has SAD 0 exactly at displacement (sx, sy)."""
+    d = synth.preset("sad", "small", seed=5)
+    sx, sy = 3, -2
+    cur = d["cur"]
+    ref = np.roll(np.roll(cur, sy, axis=0), sx, axis=1)   # ref[y+sy][x+sx] = cur[y][x]
+    s4, s8, s16 = T().sad(dict(d, ref=np.ascontiguousarray(ref)))
+    R, w, h = d["R"], d["w"], d["h"]
+    p = (sy + R) * (2 * R + 1) + (sx + R)
+    mbw = w // 16
+    inside = [mb for mb in range(s16.shape[0])
+              if 16 * (mb % mbw) + sx >= 0 and 16 * (mb % mbw) + 15 + sx < w and
+              16 * (mb // mbw) + sy >= 0 and 16 * (mb // mbw) + 15 + sy < h]
+    assert len(inside) > 50
+    assert not s16[inside, p].any() and not s4[inside, p, :].any()
