@@ -204,6 +204,21 @@ typedef struct {
   uint32_t w, h, R;
 } accel_sad_args;
 
+/* lbm -- Parboil "lbm" (D3Q19 lattice Boltzmann): launch r
+ * does one pull stream + BGK collide step from (r == 0 ? f0 : buf[(r-1)&1])
+ * into buf[r&1]; periodic boundaries, bounce-back on obstacle cells (flags
+ * != 0), velocity order and weights of oracle/tenants.c.  f arrays are SoA
+ * [19][nz][ny][nx] fp32 (DEVICE); block 128, VG = 128 cells of one x row,
+ * grid (ceil(nx/128), ny, nz). */
+typedef struct {
+  const float *f0;
+  float *buf0;
+  float *buf1;
+  const uint8_t *flags;
+  uint32_t nx, ny, nz;
+  float omega;
+} accel_lbm_args;
+
 /* mri-q ComputePhiMag: phimag = phir^2 + phii^2.  block 256, grid ceil(numk/256). */
 typedef struct {
   const float *phir;

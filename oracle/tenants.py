@@ -153,3 +153,11 @@ def sad(d: dict):
     s16 = np.empty((nmb, npos), dtype=np.uint16)
     lib().oracle_sad(_p(d["cur"]), _p(d["ref"]), I64(d["w"]), I64(d["h"]), I64(d["R"]), _p(s4), _p(s8), _p(s16))
     return s4, s8, s16
+
+
+def lbm(d: dict) -> np.ndarray:
+    """f after `steps` stream-collide steps, float64 [19][nz][ny][nx]."""
+    out = np.empty((19, d["nz"], d["ny"], d["nx"]), dtype=np.float64)
+    lib().oracle_lbm(_p(d["f0"]), _p(d["flags"]), I64(d["nx"]), I64(d["ny"]), I64(d["nz"]), I64(d["steps"]),
+                     C.c_double(d["omega"]), _p(out))
+    return out

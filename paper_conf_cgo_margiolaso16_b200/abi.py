@@ -162,6 +162,11 @@ accel_stencil_deep_args = accel_stencil_args
 accel_histo_wide_args = accel_histo_args
 
 
+class accel_lbm_args(C.Structure):
+    _fields_ = [("f0", vp), ("buf0", vp), ("buf1", vp), ("flags", vp), ("nx", u32), ("ny", u32), ("nz", u32),
+                ("omega", f32)]
+
+
 class accel_sad_args(C.Structure):
     _fields_ = [("cur", vp), ("ref", vp), ("sad4", vp), ("sad8", vp), ("sad16", vp), ("w", u32), ("h", u32), ("R", u32)]
 

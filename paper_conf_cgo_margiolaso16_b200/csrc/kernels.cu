@@ -13,6 +13,7 @@
 #include "tenants/mop.cuh"
 #include "tenants/mriq.cuh"
 #include "tenants/sad.cuh"
+#include "tenants/lbm.cuh"
 #include "tenants/sgemm.cuh"
 #include "tenants/sgemm_tc.cuh"
 #include "tenants/spmv.cuh"
@@ -122,6 +123,7 @@ const Builtin kBuiltins[] = {
     {"sgemm", &make_desc<Sgemm>},
     {"sgemm_split", &make_desc<SgemmSplit>},
     {"sgemm_tc", &make_desc<SgemmTc>},
+    {"lbm", &make_desc<Lbm>},
     {"sad_4x4", &make_desc<Sad4>},
     {"sad_8x8", &make_desc<Sad8>},
     {"sad_16x16", &make_desc<Sad16>},

@@ -70,7 +70,7 @@ struct Sad4 : SadBase {
       uint32_t s[16];
 #pragma unroll
       for (int b = 0; b < 16; ++b) s[b] = 0u;
-#pragma unroll 4
+#pragma unroll   // fully: the sub-block sums s[] must stay in registers
       for (int row = 0; row < 16; ++row) {
         const uint32_t* wr = wb + (row + dy) * kPairs;
         const uint4 c0 = *reinterpret_cast<const uint4*>(cur + row * 8);

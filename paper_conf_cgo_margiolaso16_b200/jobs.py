@@ -511,8 +511,31 @@ class SadJob(Job):
                 "skip_launches": 0, "flops_per_launch": 2.0 * 256 * n, "peak_tflops": FP32_SIMT_TFLOPS}
 
 
+class LbmJob(Job):
+    """Parboil lbm (f3): `steps` launches of the D3Q19 stream-collide step,
+    ping-pong buffers (like stencil); the result is buf[(steps-1)&1]."""
+
+    def __init__(self, d: dict, device="cuda"):
+        super().__init__(name="lbm", device=torch.device(device))
+        self.nx, self.ny, self.nz, self.nsteps = d["nx"], d["ny"], d["nz"], d["steps"]
+        n = self.nx * self.ny * self.nz
+        self.inputs = {"f0": _dev(d["f0"].ravel(), self.device), "flags": _dev(d["flags"].ravel().view(np.int8), self.device)}
+        self.buf = [torch.empty(19 * n, dtype=torch.float32, device=self.device) for _ in range(2)]
+        self.out = {"f": self.buf[(self.nsteps - 1) & 1]}
+        self.args = abi.accel_lbm_args(self.inputs["f0"].data_ptr(), self.buf[0].data_ptr(), self.buf[1].data_ptr(),
+                                       self.inputs["flags"].data_ptr(), self.nx, self.ny, self.nz, d["omega"])
+        self.steps = [Step("lbm", (_cdiv(self.nx, 128), self.ny, self.nz), self.args, self.nsteps)]
+
+    def result(self):
+        return {"f": _np(self.out["f"], np.float32).reshape(19, self.nz, self.ny, self.nx)}
+
+    def work(self):
+        b = (19 * 8 + 1) * self.nx * self.ny * self.nz
+        return {"bytes": b * self.nsteps, "bytes_per_launch": b, "bound": "hbm", "launches": self.nsteps}
+
+
 JOBS = {"mop": MopJob, "stencil": StencilJob, "histo": HistoJob, "bfs": BfsJob, "cutcp": CutcpJob,
-        "tpacf": TpacfJob, "spmv": SpmvJob, "sgemm": SgemmTcJob, "sgemm_simt": SgemmJob, "mriq": MriqJob, "sad": SadJob}
+        "tpacf": TpacfJob, "spmv": SpmvJob, "sgemm": SgemmTcJob, "sgemm_simt": SgemmJob, "mriq": MriqJob, "sad": SadJob, "lbm": LbmJob}
 
 
 def make_job(name: str, d: dict, device="cuda") -> Job:

@@ -21,6 +21,7 @@ __all__ = [
     "gen_sgemm",
     "gen_mriq",
     "gen_sad",
+    "gen_lbm",
     "GENERATORS",
 ]
 
@@ -228,8 +229,35 @@ def gen_sad(w: int, h: int, R: int = 16, seed: int = 0) -> dict:
             "w": int(w), "h": int(h), "R": int(R)}
 
 
+def gen_lbm(nx: int, ny: int, nz: int, steps: int, omega: float = 1.95, seed: int = 0) -> dict:
+    """D3Q19 lattice (SoA f[q][z][y][x] fp32) near equilibrium: rho = 1 +- 1 %,
+    u ~ U[-0.05, 0.05)^3 per cell, f = feq(rho, u) + 1e-3 w_q noise; obstacles
+    = a few seeded spheres (~5 % of the cells) [ext Parboil lbm: its obstacle
+    file is not available]."""
+    r = rng(seed)
+    c = np.array([[0, 0, 0], [1, 0, 0], [-1, 0, 0], [0, 1, 0], [0, -1, 0], [0, 0, 1], [0, 0, -1],
+                  [1, 1, 0], [-1, -1, 0], [1, -1, 0], [-1, 1, 0], [1, 0, 1], [-1, 0, -1], [1, 0, -1],
+                  [-1, 0, 1], [0, 1, 1], [0, -1, -1], [0, 1, -1], [0, -1, 1]], dtype=np.float64)
+    w = np.array([1 / 3] + [1 / 18] * 6 + [1 / 36] * 12)
+    shape = (nz, ny, nx)
+    rho = 1.0 + 0.01 * r.uniform(-1, 1, shape)
+    u = 0.05 * r.uniform(-1, 1, (3,) + shape)
+    cu = np.einsum("qd,d...->q...", c, u)
+    uu = (u * u).sum(0)
+    f = w[:, None, None, None] * rho * (1 + 3 * cu + 4.5 * cu * cu - 1.5 * uu)
+    f += 1e-3 * w[:, None, None, None] * r.uniform(-1, 1, f.shape)
+    zz, yy, xx = np.meshgrid(np.arange(nz), np.arange(ny), np.arange(nx), indexing="ij")
+    flags = np.zeros(shape, dtype=np.uint8)
+    for _ in range(max(1, (nx * ny * nz) // 40000)):
+        cz, cy, cx = r.uniform(0, nz), r.uniform(0, ny), r.uniform(0, nx)
+        rad = r.uniform(2.0, max(2.5, min(nx, ny, nz) / 8))
+        flags |= (((zz - cz) ** 2 + (yy - cy) ** 2 + (xx - cx) ** 2) < rad * rad).astype(np.uint8)
+    return {"f0": np.ascontiguousarray(f.astype(np.float32)), "flags": np.ascontiguousarray(flags),
+            "nx": int(nx), "ny": int(ny), "nz": int(nz), "steps": int(steps), "omega": float(omega)}
+
+
 GENERATORS = {
     "mop": gen_mop, "stencil": gen_stencil, "histo": gen_histo, "bfs": gen_bfs,
     "cutcp": gen_cutcp, "tpacf": gen_tpacf, "spmv": gen_spmv, "sgemm": gen_sgemm,
-    "mriq": gen_mriq, "sad": gen_sad,
+    "mriq": gen_mriq, "sad": gen_sad, "lbm": gen_lbm,
 }

@@ -60,6 +60,11 @@ PRESETS: dict[str, dict[str, dict]] = {
         "small": dict(w=176, h=144, R=16),     # QCIF
         "default": dict(w=1920, h=1072, R=16),  # [ext Parboil sad large]
     },
+    "lbm": {
+        "tiny": dict(nx=20, ny=11, nz=9, steps=3),
+        "small": dict(nx=32, ny=32, nz=32, steps=5),
+        "default": dict(nx=128, ny=128, nz=128, steps=20),   # ~2.1 M cells [ext; Parboil 120 x 120 x 150]
+    },
     "mriq": {
         "tiny": dict(nvox_1d=12, numk=300),
         "small": dict(nvox_1d=32, numk=3072),

@@ -109,3 +109,23 @@ def test_sad_default(acc, oracle_lib):
     s4, s8, s16 = oracle_lib.sad(d)
     for r in (nat, sh):
         assert np.array_equal(r["sad16"], s16) and np.array_equal(r["sad8"], s8) and np.array_equal(r["sad4"], s4)
+
+
+# ---------------------------------------------------------------- lbm (f3)
+@pytest.mark.parametrize("size,over", [("tiny", {}), ("small", {}), ("tiny", dict(nx=130, ny=5, nz=4, steps=4))])
+def test_lbm(acc_tiny_caps, oracle_lib, size, over):
+    """Parboil lbm (D3Q19 stream + BGK collide, bounce-back obstacles,
+    periodic): NATIVE == SHARED bit-exact, both within 1e-4 of the fp64 oracle."""
+    from paper_conf_cgo_margiolaso16_b200.jobs import LbmJob
+    d = synth.preset("lbm", size, **over)
+    nat, sh, _ = run_modes(acc_tiny_caps, lambda: LbmJob(d))
+    same(nat, sh)
+    assert_close_fp32(sh["f"], oracle_lib.lbm(d), what="lbm")
+
+
+def test_lbm_default(acc, oracle_lib):
+    from paper_conf_cgo_margiolaso16_b200.jobs import LbmJob
+    d = synth.preset("lbm", "default", steps=6)
+    nat, sh, _ = run_modes(acc, lambda: LbmJob(d))
+    same(nat, sh)
+    assert_close_fp32(sh["f"], oracle_lib.lbm(d), what="lbm default")

@@ -384,3 +384,54 @@ def test_sad_global_shift_is_found():
               16 * (mb // mbw) + sy >= 0 and 16 * (mb // mbw) + 15 + sy < h]
     assert len(inside) > 50
     assert not s16[inside, p].any() and not s4[inside, p, :].any()
+
+
+# ---- lbm (Parboil "lbm", D3Q19) ----------------------------
+
+_LBM_C = np.array([[0, 0, 0], [1, 0, 0], [-1, 0, 0], [0, 1, 0], [0, -1, 0], [0, 0, 1], [0, 0, -1],
+                   [1, 1, 0], [-1, -1, 0], [1, -1, 0], [-1, 1, 0], [1, 0, 1], [-1, 0, -1], [1, 0, -1],
+                   [-1, 0, 1], [0, 1, 1], [0, -1, -1], [0, 1, -1], [0, -1, 1]])
+
+
+def test_lbm_d3q19_lattice_properties():
+    """The velocity set is D3Q19 with the textbook weights: sum w = 1,
+    sum w c = 0, sum w c_a c_b = delta_ab / 3 (isotropy of the lattice)."""
+    w = np.array([1 / 3] + [1 / 18] * 6 + [1 / 36] * 12)
+    assert len({tuple(c) for c in _LBM_C}) == 19
+    assert w.sum() == pytest.approx(1.0)
+    assert np.allclose((w[:, None] * _LBM_C).sum(0), 0)
+    assert np.allclose(np.einsum("q,qa,qb->ab", w, _LBM_C, _LBM_C), np.eye(3) / 3)
+
+
+def test_lbm_conserves_mass_and_momentum():
+    """BGK collision and periodic streaming conserve mass and (without
+    obstacles) momentum; bounce-back conserves mass."""
+    d = synth.preset("lbm", "tiny", seed=2)
+    f0 = d["f0"].astype(np.float64)
+    f = T().lbm(d)
+    assert f.sum() == pytest.approx(f0.sum(), rel=1e-12)
+    dn = dict(d, flags=np.zeros_like(d["flags"]))
+    fn = T().lbm(dn)
+    mom = lambda g: _LBM_C.astype(np.float64).T @ g.reshape(19, -1).sum(axis=1)  # noqa: E731
+    assert np.allclose(mom(fn), mom(f0), rtol=0, atol=1e-9 * f0.sum())
+
+
+def test_lbm_pure_streaming_is_a_shift():
+    """omega = 0, no obstacles: one step moves every population by c_q."""
+    d = synth.preset("lbm", "tiny", seed=3)
+    d = dict(d, omega=0.0, steps=2, flags=np.zeros_like(d["flags"]))
+    f = T().lbm(d)
+    f0 = d["f0"].astype(np.float64)
+    for q, (cx, cy, cz) in enumerate(_LBM_C):
+        assert np.array_equal(f[q], np.roll(f0[q], (2 * cz, 2 * cy, 2 * cx), axis=(0, 1, 2)))
+
+
+def test_lbm_uniform_equilibrium_is_a_fixed_point():
+    d = synth.preset("lbm", "tiny", seed=4)
+    w = np.array([1 / 3] + [1 / 18] * 6 + [1 / 36] * 12)
+    rho, u = 1.02, np.array([0.03, -0.01, 0.02])
+    cu = _LBM_C @ u
+    feq = w * rho * (1 + 3 * cu + 4.5 * cu * cu - 1.5 * u @ u)
+    f0 = np.broadcast_to(feq[:, None, None, None], d["f0"].shape).astype(np.float32).copy()
+    f = T().lbm(dict(d, f0=f0, flags=np.zeros_like(d["flags"])))
+    assert np.allclose(f, f0.astype(np.float64), rtol=1e-6, atol=0)
