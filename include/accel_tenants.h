@@ -87,6 +87,24 @@ typedef struct {
   uint32_t *done;  /* [launches] */
 } accel_histo_args;
 
+/* histo_prescan / histo_intermediates -- the first two kernels of Parboil's
+ * histo pipeline, ahead of histo / histo_wide:
+ *   "histo_prescan"        lo = min raw, hi = max raw (atomicMin / atomicMax
+ *                          into *lo, *hi; the request sets *lo = 0xFFFFFFFF,
+ *                          *hi = 0 first)
+ *   "histo_intermediates"  bins_out[i] = (raw[i] - lo) * bins / (hi - lo + 1)
+ *                          (64-bit integer arithmetic), the bin index stream
+ *                          the main kernel counts
+ * block 256, VG = per_vg raw u32 samples (multiple of 1024), grid
+ * ceil(n / per_vg); raw / bins_out 16-B aligned DEVICE arrays. */
+typedef struct {
+  const uint32_t *raw;
+  uint32_t *bins_out;
+  uint32_t *lo;
+  uint32_t *hi;
+  uint32_t n, bins, per_vg;
+} accel_histo_pre_args;
+
 /* bfs -- level-synchronous top-down BFS on a directed CSR graph.
  * block 256, VG = 256 frontier vertices, static grid ceil(nv/256) (upper
  * bound; persistent CTAs read the live frontier size).  Launch l expands

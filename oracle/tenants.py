@@ -161,3 +161,14 @@ def lbm(d: dict) -> np.ndarray:
     lib().oracle_lbm(_p(d["f0"]), _p(d["flags"]), I64(d["nx"]), I64(d["ny"]), I64(d["nz"]), I64(d["steps"]),
                      C.c_double(d["omega"]), _p(out))
     return out
+
+
+def histo_pipeline(d: dict):
+    """(lo, hi, bin stream u32[n], counts u32[bins], sat u8[bins])."""
+    n, bins = d["n"], d["bins"]
+    lo, hi = C.c_uint32(), C.c_uint32()
+    bo = np.empty(n, dtype=np.uint32)
+    counts = np.empty(bins, dtype=np.uint32)
+    sat = np.empty(bins, dtype=np.uint8)
+    lib().oracle_histo_pipeline(_p(d["raw"]), I64(n), I64(bins), C.byref(lo), C.byref(hi), _p(bo), _p(counts), _p(sat))
+    return lo.value, hi.value, bo, counts, sat

@@ -162,6 +162,13 @@ accel_stencil_deep_args = accel_stencil_args
 accel_histo_wide_args = accel_histo_args
 
 
+class accel_histo_pre_args(C.Structure):
+    _fields_ = [("raw", vp), ("bins_out", vp), ("lo", vp), ("hi", vp), ("n", u32), ("bins", u32), ("per_vg", u32)]
+
+
+accel_histo_prescan_args = accel_histo_intermediates_args = accel_histo_pre_args
+
+
 class accel_lbm_args(C.Structure):
     _fields_ = [("f0", vp), ("buf0", vp), ("buf1", vp), ("flags", vp), ("nx", u32), ("ny", u32), ("nz", u32),
                 ("omega", f32)]

@@ -116,6 +116,8 @@ const Builtin kBuiltins[] = {
     {"stencil_tma", &make_desc<StencilTma>},
     {"histo", &make_desc<Histo>},
     {"histo_wide", &make_desc<HistoWide>},
+    {"histo_prescan", &make_desc<HistoPrescan>},
+    {"histo_intermediates", &make_desc<HistoIntermediates>},
     {"bfs", &make_desc<Bfs>},
     {"cutcp", &make_desc<Cutcp>},
     {"tpacf", &make_desc<Tpacf>},

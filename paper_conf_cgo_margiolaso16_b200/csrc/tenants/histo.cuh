@@ -120,6 +120,78 @@ struct HistoT {
   }
 };
 
+// Parboil histo's first two kernels: the input range and
+// the bin-index stream.  Both stream the raw samples with 16-B loads (HBM).
+struct HistoPrescan {
+  using Args = accel_histo_pre_args;
+  static constexpr int kThreads = 256;
+  static constexpr uint32_t kChunk = 1;
+  static constexpr int kMinBlocks = 6;
+  static constexpr uint32_t kDynSmem = 0;
+  static __device__ __forceinline__ void body(const Args& a, const VirtualBlock& vb, char*) {
+    __shared__ uint32_t s_lo[kThreads / 32], s_hi[kThreads / 32];
+    const uint64_t lo0 = (uint64_t)vb.linear * a.per_vg;
+    const uint64_t hi0 = lo0 + a.per_vg < a.n ? lo0 + a.per_vg : a.n;
+    uint32_t mn = 0xffffffffu, mx = 0u;
+    const uint64_t nvec = (hi0 - lo0) / 4;
+    const uint4* v = reinterpret_cast<const uint4*>(a.raw + lo0);
+    for (uint64_t i = threadIdx.x; i < nvec; i += kThreads) {
+      const uint4 w = __ldcs(v + i);
+      mn = min(min(mn, w.x), min(w.y, min(w.z, w.w)));
+      mx = max(max(mx, w.x), max(w.y, max(w.z, w.w)));
+    }
+    for (uint64_t i = lo0 + nvec * 4 + threadIdx.x; i < hi0; i += kThreads) {
+      mn = min(mn, a.raw[i]);
+      mx = max(mx, a.raw[i]);
+    }
+    mn = __reduce_min_sync(0xffffffffu, mn);
+    mx = __reduce_max_sync(0xffffffffu, mx);
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    if (lane == 0) {
+      s_lo[warp] = mn;
+      s_hi[warp] = mx;
+    }
+    __syncthreads();
+    if (threadIdx.x < 32) {
+      mn = lane < kThreads / 32 ? s_lo[lane] : 0xffffffffu;
+      mx = lane < kThreads / 32 ? s_hi[lane] : 0u;
+      mn = __reduce_min_sync(0xffffffffu, mn);
+      mx = __reduce_max_sync(0xffffffffu, mx);
+      if (lane == 0) {
+        atomicMin(a.lo, mn);
+        atomicMax(a.hi, mx);
+      }
+    }
+    __syncthreads();   // s_lo / s_hi are reused by the CTA's next VG
+  }
+};
+
+struct HistoIntermediates {
+  using Args = accel_histo_pre_args;
+  static constexpr int kThreads = 256;
+  static constexpr uint32_t kChunk = 1;
+  static constexpr int kMinBlocks = 6;
+  static constexpr uint32_t kDynSmem = 0;
+  static __device__ __forceinline__ uint32_t bin(uint32_t x, uint32_t lo, uint64_t span, uint32_t bins) {
+    return (uint32_t)(((uint64_t)(x - lo) * bins) / span);
+  }
+  static __device__ __forceinline__ void body(const Args& a, const VirtualBlock& vb, char*) {
+    const uint32_t lo = __ldcg(a.lo), hi = __ldcg(a.hi), bins = a.bins;
+    const uint64_t span = (uint64_t)(hi - lo) + 1u;
+    const uint64_t lo0 = (uint64_t)vb.linear * a.per_vg;
+    const uint64_t hi0 = lo0 + a.per_vg < a.n ? lo0 + a.per_vg : a.n;
+    const uint64_t nvec = (hi0 - lo0) / 4;
+    const uint4* v = reinterpret_cast<const uint4*>(a.raw + lo0);
+    uint4* o = reinterpret_cast<uint4*>(a.bins_out + lo0);
+    for (uint64_t i = threadIdx.x; i < nvec; i += kThreads) {
+      const uint4 w = __ldcs(v + i);
+      o[i] = make_uint4(bin(w.x, lo, span, bins), bin(w.y, lo, span, bins), bin(w.z, lo, span, bins),
+                        bin(w.w, lo, span, bins));
+    }
+    for (uint64_t i = lo0 + nvec * 4 + threadIdx.x; i < hi0; i += kThreads) a.bins_out[i] = bin(a.raw[i], lo, span, bins);
+  }
+};
+
 using Histo = HistoT<false>;
 using HistoWide = HistoT<true>;
 

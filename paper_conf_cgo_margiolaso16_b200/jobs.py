@@ -217,7 +217,9 @@ class StencilJob(Job):
 
 
 class HistoJob(Job):
-    def __init__(self, d: dict, device="cuda"):
+    def __init__(self, d: dict, device="cuda", samples: torch.Tensor | None = None):
+        """samples: an existing device stream of bin indices (the histo
+        pipeline's intermediates) instead of d["samples"]."""
         super().__init__(name="histo", device=torch.device(device))
         self.n, self.bins, self.iters, self.sb = d["n"], d["bins"], d["iters"], d["sample_bytes"]
         if not (1 <= self.bins <= 16384 and (self.sb == 4 or self.bins == 256)):
@@ -229,13 +231,14 @@ class HistoJob(Job):
         # (measured at the SURVEY default: 74 -> 52 us per pass, 16384 -> 61440)
         self.per_vg = 4096 if self.sb == 1 else d.get("per_vg", 16384 if self.kernel == "histo" else 61440)
         assert self.per_vg % 4096 == 0 and (self.kernel == "histo" or self.per_vg < 65536)
-        self.inputs = {"samples": _dev(d["samples"], self.device)}
+        self.inputs = {"samples": _dev(d["samples"], self.device)} if samples is None else {}
+        src = samples if samples is not None else self.inputs["samples"]
         self.hist = torch.zeros(2 * self.bins, dtype=torch.int32, device=self.device)
         self.sat = torch.zeros(self.bins, dtype=torch.uint8, device=self.device)
         self.done = torch.zeros(self.iters, dtype=torch.int32, device=self.device)
         last = (self.iters - 1) & 1
         self.out = {"counts": self.hist[last * self.bins:(last + 1) * self.bins], "sat": self.sat}
-        self.args = abi.accel_histo_args(self.inputs["samples"].data_ptr(), self.n, self.bins, self.sb,
+        self.args = abi.accel_histo_args(src.data_ptr(), self.n, self.bins, self.sb,
                                          self.per_vg, self.hist.data_ptr(), self.sat.data_ptr(),
                                          self.done.data_ptr())
         self.clears = [(self.hist, 0), (self.done, 0)]
@@ -511,6 +514,43 @@ class SadJob(Job):
                 "skip_launches": 0, "flops_per_launch": 2.0 * 256 * n, "peak_tflops": FP32_SIMT_TFLOPS}
 
 
+class HistoPipelineJob(Job):
+    """Parboil histo's whole pipeline (f3): prescan (input range), intermediates
+    (raw samples -> bin indices), then `iters` launches of the main+final
+    kernel on the bin stream -- one request, three steps (main = the last)."""
+
+    PER_VG = 16384
+
+    def __init__(self, d: dict, device="cuda"):
+        super().__init__(name="histo_pipeline", device=torch.device(device))
+        self.n, self.bins, self.iters = d["n"], d["bins"], d["iters"]
+        self.inputs = {"raw": _dev(d["raw"], self.device)}
+        self.bin_stream = torch.empty(self.n, dtype=torch.int32, device=self.device)
+        self.lo = torch.empty(1, dtype=torch.int32, device=self.device)
+        self.hi = torch.empty(1, dtype=torch.int32, device=self.device)
+        self.main = HistoJob({"n": self.n, "bins": self.bins, "iters": self.iters, "sample_bytes": 4,
+                              "samples": np.zeros(0, dtype=np.uint32)}, device, samples=self.bin_stream)
+        self.hist, self.sat = self.main.hist, self.main.sat
+        self.out = dict(self.main.out, lo=self.lo, hi=self.hi)
+        self.args_pre = abi.accel_histo_pre_args(self.inputs["raw"].data_ptr(), self.bin_stream.data_ptr(),
+                                                 self.lo.data_ptr(), self.hi.data_ptr(), self.n, self.bins,
+                                                 self.PER_VG)
+        self.clears = [(self.lo, 0xFF), (self.hi, 0)] + self.main.clears
+        g = (_cdiv(self.n, self.PER_VG), 1, 1)
+        self.main_step = 2
+        self.steps = [Step("histo_prescan", g, self.args_pre, 1), Step("histo_intermediates", g, self.args_pre, 1),
+                      self.main.steps[0]]
+
+    def result(self):
+        r = self.main.result()
+        r.update(lo=int(_np(self.lo, np.uint32)[0]), hi=int(_np(self.hi, np.uint32)[0]))
+        return r
+
+    def work(self):
+        b = 4 * self.n
+        return {"bytes": 3 * b + self.main.work()["bytes"], "bound": "hbm", "launches": 2 + self.iters}
+
+
 class LbmJob(Job):
     """Parboil lbm (f3): `steps` launches of the D3Q19 stream-collide step,
     ping-pong buffers (like stencil); the result is buf[(steps-1)&1]."""
@@ -535,7 +575,8 @@ class LbmJob(Job):
 
 
 JOBS = {"mop": MopJob, "stencil": StencilJob, "histo": HistoJob, "bfs": BfsJob, "cutcp": CutcpJob,
-        "tpacf": TpacfJob, "spmv": SpmvJob, "sgemm": SgemmTcJob, "sgemm_simt": SgemmJob, "mriq": MriqJob, "sad": SadJob, "lbm": LbmJob}
+        "tpacf": TpacfJob, "spmv": SpmvJob, "sgemm": SgemmTcJob, "sgemm_simt": SgemmJob, "mriq": MriqJob, "sad": SadJob, "lbm": LbmJob,
+        "histo_pipeline": HistoPipelineJob}
 
 
 def make_job(name: str, d: dict, device="cuda") -> Job:

@@ -22,6 +22,7 @@ __all__ = [
     "gen_mriq",
     "gen_sad",
     "gen_lbm",
+    "gen_histo_raw",
     "GENERATORS",
 ]
 
@@ -256,8 +257,20 @@ def gen_lbm(nx: int, ny: int, nz: int, steps: int, omega: float = 1.95, seed: in
             "nx": int(nx), "ny": int(ny), "nz": int(nz), "steps": int(steps), "omega": float(omega)}
 
 
+def gen_histo_raw(n: int, bins: int, iters: int, seed: int = 0) -> dict:
+    """Raw u32 samples for Parboil histo's full pipeline: the skewed bin
+    distribution of gen_histo, scaled by 4096, plus a uniform in-bin offset
+    and a seeded base (the prescan finds the range, the intermediates map it
+    back to bins)."""
+    r = rng(seed)
+    s = gen_histo(n, bins, iters, 4, seed)["samples"].astype(np.uint64)
+    base = int(r.integers(1_000, 1_000_000))
+    raw = base + s * 4096 + r.integers(0, 4096, n, dtype=np.uint64)
+    return {"raw": np.ascontiguousarray(raw.astype(np.uint32)), "n": int(n), "bins": int(bins), "iters": int(iters)}
+
+
 GENERATORS = {
     "mop": gen_mop, "stencil": gen_stencil, "histo": gen_histo, "bfs": gen_bfs,
     "cutcp": gen_cutcp, "tpacf": gen_tpacf, "spmv": gen_spmv, "sgemm": gen_sgemm,
-    "mriq": gen_mriq, "sad": gen_sad, "lbm": gen_lbm,
+    "mriq": gen_mriq, "sad": gen_sad, "lbm": gen_lbm, "histo_pipeline": gen_histo_raw,
 }

@@ -60,6 +60,11 @@ PRESETS: dict[str, dict[str, dict]] = {
         "small": dict(w=176, h=144, R=16),     # QCIF
         "default": dict(w=1920, h=1072, R=16),  # [ext Parboil sad large]
     },
+    "histo_pipeline": {
+        "tiny": dict(n=100_003, bins=16384, iters=2),
+        "small": dict(n=1 << 18, bins=4096, iters=3),
+        "default": dict(n=1 << 24, bins=16384, iters=20),
+    },
     "lbm": {
         "tiny": dict(nx=20, ny=11, nz=9, steps=3),
         "small": dict(nx=32, ny=32, nz=32, steps=5),

@@ -347,3 +347,25 @@ def test_tpacf_qsplit(acc_tiny_caps, oracle_lib, qsplit):
     dd, rr, dr = oracle_lib.tpacf(d)
     for r in (nat, sh):
         assert np.array_equal(r["dd"], dd) and np.array_equal(r["rr"], rr) and np.array_equal(r["dr"], dr)
+
+
+@pytest.mark.parametrize("size", ["tiny", "small"])
+def test_histo_pipeline(acc_tiny_caps, oracle_lib, size):
+    """Parboil histo's full pipeline (f3): prescan range and intermediate bin
+    stream, then the histogram -- bit-exact in both modes."""
+    from paper_conf_cgo_margiolaso16_b200.jobs import HistoPipelineJob
+    d = synth.preset("histo_pipeline", size)
+    lo, hi, bo, counts, sat = oracle_lib.histo_pipeline(d)
+    nat, sh, _ = run_modes(acc_tiny_caps, lambda: HistoPipelineJob(d))
+    for r in (nat, sh):
+        assert (r["lo"], r["hi"]) == (lo, hi)
+        assert np.array_equal(r["counts"], counts) and np.array_equal(r["sat"], sat)
+
+
+def test_histo_pipeline_default(acc, oracle_lib):
+    from paper_conf_cgo_margiolaso16_b200.jobs import HistoPipelineJob
+    d = synth.preset("histo_pipeline", "default", iters=3)
+    lo, hi, bo, counts, sat = oracle_lib.histo_pipeline(d)
+    nat, sh, _ = run_modes(acc, lambda: HistoPipelineJob(d))
+    for r in (nat, sh):
+        assert (r["lo"], r["hi"]) == (lo, hi) and np.array_equal(r["counts"], counts)

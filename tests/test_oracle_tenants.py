@@ -435,3 +435,29 @@ def test_lbm_uniform_equilibrium_is_a_fixed_point():
     f0 = np.broadcast_to(feq[:, None, None, None], d["f0"].shape).astype(np.float32).copy()
     f = T().lbm(dict(d, f0=f0, flags=np.zeros_like(d["flags"])))
     assert np.allclose(f, f0.astype(np.float64), rtol=1e-6, atol=0)
+
+
+# ---- histo pipeline: prescan + intermediates (Parboil histo; f3) ------------
+
+def test_histo_pipeline_numpy():
+    d = synth.preset("histo_pipeline", "tiny", seed=6)
+    lo, hi, bo, counts, sat = T().histo_pipeline(d)
+    raw = d["raw"].astype(np.uint64)
+    assert lo == raw.min() and hi == raw.max()
+    ref = ((raw - lo) * d["bins"]) // (hi - lo + 1)
+    assert np.array_equal(bo, ref.astype(np.uint32))
+    assert np.array_equal(counts, np.bincount(ref, minlength=d["bins"]).astype(np.uint32))
+    assert int(counts.sum()) == d["n"] and bo.max() < d["bins"]
+    assert np.array_equal(sat, np.minimum(counts, 255).astype(np.uint8))
+
+
+def test_histo_pipeline_recovers_the_bins():
+    """raw = base + 4096 * s + U[0, 4096): when the extreme bins are both hit,
+    the intermediates map (almost) every sample back to its generating bin s
+    (lo and hi sit within one bin width of base and base + 4096 * bins, so
+    only samples within that slack of a bin edge move)."""
+    d = synth.preset("histo_pipeline", "small", seed=7)
+    _, _, bo, _, _ = T().histo_pipeline(d)
+    s = gen.gen_histo(d["n"], d["bins"], d["iters"], 4, 7)["samples"]
+    if s.min() == 0 and s.max() == d["bins"] - 1:
+        assert np.mean(bo == s) > 0.99 and np.all(np.abs(bo.astype(np.int64) - s) <= 1)
