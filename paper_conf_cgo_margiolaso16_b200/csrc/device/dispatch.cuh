@@ -412,14 +412,16 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     // CTAs on one queue word serialised in L2 and spread the CTAs' first VG
     // starts over 6 us of a 30-us stencil launch (scripts/vg_trace.py)
     const bool stat = (cfg & kCfgStaticFirst) != 0u;
+    uint32_t topped_prev = 0;
     if (!kResolve) {
       b = stat ? blockIdx.x * chunk : qa_next(atomicAdd(&d->qa, (unsigned long long)chunk));
     } else {
       // a predecessor launch that was topped up may still be running on its
       // top-up CTAs: this grid's body must wait for it.  The flag load, the
-      // admission and the first dequeue are all issued before the wait, so a
-      // launch that was never topped pays no extra round trip
-      const uint32_t topped_prev =
+      // admission, the first dequeue and the scheduling-state set-up are all
+      // issued before the flag is tested, so a launch that was never topped
+      // pays no serial round trip for it
+      topped_prev =
           (cfg & kCfgWaitPrev) ? 1u
           : ((cfg & kCfgHasPrev) && !(cfg & kAblNoTop)) ? ld_volatile(&(d - 1)->topped) : 0u;
       // admission and first dequeue in one atomic; an arrival over the live
@@ -452,10 +454,15 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
       if (b == 0) asm volatile("red.relaxed.gpu.global.max.u32 [%0], %1;" ::"l"(&d->ctl->cur), "r"(d->req_idx) : "memory");
       S->hint_live = live;
       S->hint_alive = a;
-      if (topped_prev) wait_complete(d - 1);
     }
-    if (cfg & kCfgStamps) red_min_u64(&d->t_first, globaltimer());
     const uint32_t launch_idx = d->launch_idx;
+    // a dynamic total is the predecessor's output: read it after the wait
+    if constexpr (has_dynamic_total<T>::value) {
+      if (topped_prev) {
+        wait_complete(d - 1);
+        topped_prev = 0;
+      }
+    }
     const uint32_t total = vg_total<T>(args, d, launch_idx);
     // RESOLVE: every CTA publishes the total (the same value: a
     // dynamic total is final once the predecessor launch completed).  Top-up
@@ -479,6 +486,8 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     S->spread = has_spread<T>::value ? spread_factor(total) : 0u;
     S->prefetch_window = 2u * chunk * gridDim.x;
     S->template set_cur<has_spread<T>::value>(0, b);
+    if (topped_prev) wait_complete(d - 1);
+    if (cfg & kCfgStamps) red_min_u64(&d->t_first, globaltimer());
   }
   __syncthreads();
   // thread 0: the prefetched queue word and live quota stay in registers
