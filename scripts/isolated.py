@@ -58,9 +58,17 @@ def main():
                 acc.release()
             el, lt = el[1:], lt[1:]
             w = job.work()
-            per = [x for l in lt for x in l]
+            # per-launch times of the MAIN step only (the GEMM, not its operand
+            # split; mri-q's Q, not PhiMag): the roofline is that kernel's
+            first = sum(st.repeat for st in job.steps[:job.main_step]) if job.main_step >= 0 else 0
+            nmain = job.steps[job.main_step].repeat if job.main_step >= 0 else job.launches()
+            per = [x for l in lt for x in l[first:first + nmain]]
+            by_step, k = [], 0
+            for st in job.steps:
+                by_step.append(statistics.mean(x for l in lt for x in l[k:k + st.repeat]))
+                k += st.repeat
             r = {"elapsed_ms": statistics.median(el), "launch_ms_mean": statistics.mean(per),
-                 "launch_ms_min": min(per), "quota": q}
+                 "launch_ms_min": min(per), "launch_ms_by_step": by_step, "quota": q}
             if w.get("bound") == "hbm":
                 b = w.get("bytes_per_launch", w.get("bytes"))
                 r["GBps_mean"] = b / r["launch_ms_mean"] / 1e6
