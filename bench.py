@@ -577,7 +577,11 @@ def main(argv=None):
                 cpu = {"value": None, "unit": UNIT, "cores": os.cpu_count(), "kind": "oracle", "sample": "stub"}
             else:
                 cpu = cpu_baseline(local_res["tenants"], inputs)
-        print(json.dumps(result_line(args, allres, world, cpu)), flush=True)
+        line = json.dumps(result_line(args, allres, world, cpu))
+        print(line, flush=True)
+        if args.out:
+            with open(args.out, "w") as f:
+                f.write(line + "\n")
     ranks.barrier()
     ranks.close()
     return 0

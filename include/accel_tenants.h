@@ -237,6 +237,37 @@ typedef struct {
   float omega;
 } accel_lbm_args;
 
+/* mri-gridding -- Parboil "mri-gridding": non-Cartesian
+ * samples convolved onto a G^3 grid with a separable Kaiser-Bessel kernel
+ * (definition: oracle/tenants.c oracle_gridding).  Six kernels, the six steps
+ * of one request, all with this argument struct:
+ *   "gridding_binning"    VG = 1024 samples: bin[i] = cell of sample i (cells
+ *                         of `cell` grid units), rank[i] = atomicAdd(count[bin])
+ *   "gridding_scan_l1"    VG = 1024 bins: start[b] = exclusive scan within the
+ *                         VG, block_sum[vg] = its total
+ *   "gridding_scan_inter" 1 VG: exclusive scan of block_sum, start[B] = n
+ *   "gridding_scan_add"   VG = 1024 bins: start[b] += block_sum[vg]
+ *   "gridding_reorder"    VG = 1024 samples: the samples in bin order
+ *   "gridding_grid"       VG = 8 x 8 x 8 grid points (256 threads, 2 points
+ *                         each): the samples of the bins within hw of the
+ *                         tile, per-point sums in 64-bit fixed point (2^-30:
+ *                         order-independent, so NATIVE and SHARED agree bit
+ *                         for bit whatever order the binning's atomics chose),
+ *                         grid[p] = (re, im) fp32
+ * B = cells^3 <= 1024 * 1024; count cleared by the request; DEVICE buffers. */
+typedef struct {
+  const float *x, *y, *z, *re, *im;   /* input samples [n] */
+  const float *lut;                   /* [L] Kaiser-Bessel table */
+  uint32_t L, n, G, cells;            /* cells per dimension = ceil(G / cell) */
+  float hw, cell;                     /* kernel half-width, cell edge (grid units) */
+  uint32_t *bin, *rank;               /* [n] */
+  uint32_t *count;                    /* [B] */
+  uint32_t *start;                    /* [B + 1] */
+  uint32_t *block_sum;                /* [ceil(B / 1024)] */
+  float *sx, *sy, *sz, *sre, *sim;    /* [n] in bin order */
+  float *grid;                        /* [G][G][G][2] */
+} accel_gridding_args;
+
 /* mri-q ComputePhiMag: phimag = phir^2 + phii^2.  block 256, grid ceil(numk/256). */
 typedef struct {
   const float *phir;

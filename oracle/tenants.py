@@ -172,3 +172,12 @@ def histo_pipeline(d: dict):
     sat = np.empty(bins, dtype=np.uint8)
     lib().oracle_histo_pipeline(_p(d["raw"]), I64(n), I64(bins), C.byref(lo), C.byref(hi), _p(bo), _p(counts), _p(sat))
     return lo.value, hi.value, bo, counts, sat
+
+
+def gridding(d: dict) -> np.ndarray:
+    """grid complex [G][G][G][2] float64 (re, im)."""
+    G = d["G"]
+    g = np.empty((G, G, G, 2), dtype=np.float64)
+    lib().oracle_gridding(_p(d["x"]), _p(d["y"]), _p(d["z"]), _p(d["re"]), _p(d["im"]), I64(d["n"]), I64(G),
+                          C.c_float(d["hw"]), _p(d["lut"]), I64(len(d["lut"])), _p(g))
+    return g

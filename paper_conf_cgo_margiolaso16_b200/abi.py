@@ -169,6 +169,17 @@ class accel_histo_pre_args(C.Structure):
 accel_histo_prescan_args = accel_histo_intermediates_args = accel_histo_pre_args
 
 
+class accel_gridding_args(C.Structure):
+    _fields_ = [("x", vp), ("y", vp), ("z", vp), ("re", vp), ("im", vp), ("lut", vp),
+                ("L", u32), ("n", u32), ("G", u32), ("cells", u32), ("hw", f32), ("cell", f32),
+                ("bin", vp), ("rank", vp), ("count", vp), ("start", vp), ("block_sum", vp),
+                ("sx", vp), ("sy", vp), ("sz", vp), ("sre", vp), ("sim", vp), ("grid", vp)]
+
+
+accel_gridding_binning_args = accel_gridding_scan_l1_args = accel_gridding_scan_inter_args = accel_gridding_args
+accel_gridding_scan_add_args = accel_gridding_reorder_args = accel_gridding_grid_args = accel_gridding_args
+
+
 class accel_lbm_args(C.Structure):
     _fields_ = [("f0", vp), ("buf0", vp), ("buf1", vp), ("flags", vp), ("nx", u32), ("ny", u32), ("nz", u32),
                 ("omega", f32)]

@@ -14,6 +14,7 @@
 #include "tenants/mriq.cuh"
 #include "tenants/sad.cuh"
 #include "tenants/lbm.cuh"
+#include "tenants/gridding.cuh"
 #include "tenants/sgemm.cuh"
 #include "tenants/sgemm_tc.cuh"
 #include "tenants/spmv.cuh"
@@ -126,6 +127,12 @@ const Builtin kBuiltins[] = {
     {"sgemm_split", &make_desc<SgemmSplit>},
     {"sgemm_tc", &make_desc<SgemmTc>},
     {"lbm", &make_desc<Lbm>},
+    {"gridding_binning", &make_desc<GridBinning>},
+    {"gridding_scan_l1", &make_desc<GridScanL1>},
+    {"gridding_scan_inter", &make_desc<GridScanInter>},
+    {"gridding_scan_add", &make_desc<GridScanAdd>},
+    {"gridding_reorder", &make_desc<GridReorder>},
+    {"gridding_grid", &make_desc<GridGrid>},
     {"sad_4x4", &make_desc<Sad4>},
     {"sad_8x8", &make_desc<Sad8>},
     {"sad_16x16", &make_desc<Sad16>},

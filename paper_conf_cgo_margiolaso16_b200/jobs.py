@@ -551,6 +551,50 @@ class HistoPipelineJob(Job):
         return {"bytes": 3 * b + self.main.work()["bytes"], "bound": "hbm", "launches": 2 + self.iters}
 
 
+class GriddingJob(Job):
+    """Parboil mri-gridding (f3): six steps -- binning, the three-kernel scan
+    of the cell counts, reorder, gridding -- one request (main = gridding)."""
+
+    CELL = 2.0   # cell edge in grid units: the gridding VG reads the cells within hw of its 8^3 tile
+
+    def __init__(self, d: dict, device="cuda"):
+        super().__init__(name="gridding", device=torch.device(device))
+        self.n, self.G, self.hw = d["n"], d["G"], d["hw"]
+        dev = self.device
+        self.inputs = {k: _dev(d[k], dev) for k in ("x", "y", "z", "re", "im", "lut")}
+        self.cells = _cdiv(self.G, int(self.CELL))
+        B = self.cells ** 3
+        if B > 1024 * 1024 or len(d["lut"]) > 1024:
+            raise ValueError("gridding: at most 1024^2 cells and 1024 LUT entries")
+        u32 = lambda m: torch.empty(m, dtype=torch.int32, device=dev)  # noqa: E731
+        f32 = lambda m: torch.empty(m, dtype=torch.float32, device=dev)  # noqa: E731
+        self.bin, self.rank, self.count, self.start = u32(self.n), u32(self.n), u32(B), u32(B + 1)
+        self.block_sum = u32(_cdiv(B, 1024))
+        self.sorted = [f32(self.n) for _ in range(5)]
+        self.grid = f32(2 * self.G ** 3)
+        self.out = {"grid": self.grid}
+        i = self.inputs
+        self.args = abi.accel_gridding_args(i["x"].data_ptr(), i["y"].data_ptr(), i["z"].data_ptr(),
+                                            i["re"].data_ptr(), i["im"].data_ptr(), i["lut"].data_ptr(),
+                                            len(d["lut"]), self.n, self.G, self.cells, self.hw, self.CELL,
+                                            self.bin.data_ptr(), self.rank.data_ptr(), self.count.data_ptr(),
+                                            self.start.data_ptr(), self.block_sum.data_ptr(),
+                                            *[t.data_ptr() for t in self.sorted], self.grid.data_ptr())
+        self.clears = [(self.count, 0)]
+        gs, gb = (_cdiv(self.n, 1024), 1, 1), (_cdiv(B, 1024), 1, 1)
+        t = _cdiv(self.G, 8)
+        self.main_step = 5
+        self.steps = [Step("gridding_binning", gs, self.args), Step("gridding_scan_l1", gb, self.args),
+                      Step("gridding_scan_inter", (1, 1, 1), self.args), Step("gridding_scan_add", gb, self.args),
+                      Step("gridding_reorder", gs, self.args), Step("gridding_grid", (t, t, t), self.args)]
+
+    def result(self):
+        return {"grid": _np(self.grid, np.float32).reshape(self.G, self.G, self.G, 2)}
+
+    def work(self):
+        return {"bytes": 4 * 8 * self.G ** 3 + 20 * self.n, "bound": "alu", "launches": 6}
+
+
 class LbmJob(Job):
     """Parboil lbm (f3): `steps` launches of the D3Q19 stream-collide step,
     ping-pong buffers (like stencil); the result is buf[(steps-1)&1]."""
@@ -576,7 +620,7 @@ class LbmJob(Job):
 
 JOBS = {"mop": MopJob, "stencil": StencilJob, "histo": HistoJob, "bfs": BfsJob, "cutcp": CutcpJob,
         "tpacf": TpacfJob, "spmv": SpmvJob, "sgemm": SgemmTcJob, "sgemm_simt": SgemmJob, "mriq": MriqJob, "sad": SadJob, "lbm": LbmJob,
-        "histo_pipeline": HistoPipelineJob}
+        "histo_pipeline": HistoPipelineJob, "gridding": GriddingJob}
 
 
 def make_job(name: str, d: dict, device="cuda") -> Job:

@@ -23,6 +23,7 @@ __all__ = [
     "gen_sad",
     "gen_lbm",
     "gen_histo_raw",
+    "gen_gridding",
     "GENERATORS",
 ]
 
@@ -269,8 +270,35 @@ def gen_histo_raw(n: int, bins: int, iters: int, seed: int = 0) -> dict:
     return {"raw": np.ascontiguousarray(raw.astype(np.uint32)), "n": int(n), "bins": int(bins), "iters": int(iters)}
 
 
+def gen_gridding(G: int, n: int, W: float = 4.0, L: int = 1024, seed: int = 0) -> dict:
+    """MRI k-space samples for gridding [ext Parboil mri-gridding]: n points on
+    a few radial-ish spokes plus uniform jitter inside [0, G)^3 (denser near
+    the centre, like a radial acquisition), complex values U[-1, 1)^2; the
+    separable Kaiser-Bessel kernel of width W (half-width W/2) tabulated at L
+    points, beta = pi sqrt((W/2)^2 (2 - 0.5)^2 - 0.8) (oversampling 2),
+    normalised to 1 at distance 0 -- computed here in fp64."""
+    r = rng(seed)
+    hw = W / 2.0
+    c = G / 2.0
+    t = r.uniform(-1, 1, n) ** 3                      # denser near the centre
+    dirs = r.normal(0, 1, (64, 3))
+    dirs /= np.linalg.norm(dirs, axis=1, keepdims=True)
+    pick = dirs[r.integers(0, 64, n)]
+    pts = c + (G / 2.0 - hw) * t[:, None] * pick + r.normal(0, 1.5, (n, 3))
+    pts = np.clip(pts, 0.0, np.nextafter(G, 0))
+    beta = np.pi * np.sqrt((W / 2.0) ** 2 * (2.0 - 0.5) ** 2 - 0.8)
+    dist = np.arange(L) * hw / (L - 1)
+    arg = beta * np.sqrt(np.maximum(0.0, 1.0 - (dist / hw) ** 2))
+    lut = np.i0(arg) / np.i0(beta)
+    return {"x": np.ascontiguousarray(pts[:, 0].astype(np.float32)), "y": np.ascontiguousarray(pts[:, 1].astype(np.float32)),
+            "z": np.ascontiguousarray(pts[:, 2].astype(np.float32)),
+            "re": r.uniform(-1, 1, n).astype(np.float32), "im": r.uniform(-1, 1, n).astype(np.float32),
+            "lut": lut.astype(np.float32), "n": int(n), "G": int(G), "hw": float(hw)}
+
+
 GENERATORS = {
     "mop": gen_mop, "stencil": gen_stencil, "histo": gen_histo, "bfs": gen_bfs,
     "cutcp": gen_cutcp, "tpacf": gen_tpacf, "spmv": gen_spmv, "sgemm": gen_sgemm,
     "mriq": gen_mriq, "sad": gen_sad, "lbm": gen_lbm, "histo_pipeline": gen_histo_raw,
+    "gridding": gen_gridding,
 }

@@ -65,6 +65,11 @@ PRESETS: dict[str, dict[str, dict]] = {
         "small": dict(n=1 << 18, bins=4096, iters=3),
         "default": dict(n=1 << 24, bins=16384, iters=20),
     },
+    "gridding": {
+        "tiny": dict(G=24, n=3000),
+        "small": dict(G=48, n=40000),
+        "default": dict(G=128, n=1 << 20),
+    },
     "lbm": {
         "tiny": dict(nx=20, ny=11, nz=9, steps=3),
         "small": dict(nx=32, ny=32, nz=32, steps=5),

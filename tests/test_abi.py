@@ -59,7 +59,7 @@ def test_struct_layouts_match_c(tmp_path):
                "accel_histo_args", "accel_bfs_args", "accel_cutcp_args", "accel_tpacf_args",
                "accel_spmv_args", "accel_sgemm_args", "accel_sgemm_split_args", "accel_sgemm_tc_args",
                "accel_mriq_phimag_args", "accel_mriq_q_args", "accel_stencil_tma_args", "accel_sad_args",
-               "accel_lbm_args", "accel_histo_pre_args"]
+               "accel_lbm_args", "accel_histo_pre_args", "accel_gridding_args"]
     src = tmp_path / "s.c"
     src.write_text('#include <stdio.h>\n#include "accel.h"\n#include "accel_tenants.h"\nint main(){\n' +
                    "".join(f'printf("%zu\\n", sizeof({s}));\n' for s in structs) + "return 0;}\n")

@@ -129,3 +129,24 @@ def test_lbm_default(acc, oracle_lib):
     nat, sh, _ = run_modes(acc, lambda: LbmJob(d))
     same(nat, sh)
     assert_close_fp32(sh["f"], oracle_lib.lbm(d), what="lbm default")
+
+
+# ---------------------------------------------------------------- mri-gridding (f3)
+@pytest.mark.parametrize("size,over", [("tiny", {}), ("small", {}), ("tiny", dict(G=21, n=5000))])
+def test_gridding(acc_tiny_caps, oracle_lib, size, over):
+    """Parboil mri-gridding pipeline (binning, 3-kernel scan, reorder,
+    gridding): NATIVE == SHARED bit-exact (fixed-point sums: independent of
+    the atomic binning order), within 1e-4 of the fp64 oracle."""
+    from paper_conf_cgo_margiolaso16_b200.jobs import GriddingJob
+    d = synth.preset("gridding", size, **over)
+    nat, sh, _ = run_modes(acc_tiny_caps, lambda: GriddingJob(d))
+    same(nat, sh)
+    assert_close_fp32(sh["grid"], oracle_lib.gridding(d), what="gridding")
+
+
+def test_gridding_default(acc, oracle_lib):
+    from paper_conf_cgo_margiolaso16_b200.jobs import GriddingJob
+    d = synth.preset("gridding", "default")
+    nat, sh, _ = run_modes(acc, lambda: GriddingJob(d))
+    same(nat, sh)
+    assert_close_fp32(sh["grid"], oracle_lib.gridding(d), what="gridding default")

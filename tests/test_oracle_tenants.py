@@ -461,3 +461,54 @@ def test_histo_pipeline_recovers_the_bins():
     s = gen.gen_histo(d["n"], d["bins"], d["iters"], 4, 7)["samples"]
     if s.min() == 0 and s.max() == d["bins"] - 1:
         assert np.mean(bo == s) > 0.99 and np.all(np.abs(bo.astype(np.int64) - s) <= 1)
+
+
+# ---- mri-gridding (Parboil) --------------------------------
+
+def _gridding_numpy(d):
+    """numpy brute force: every (grid point, sample) pair, the fp32 index
+    decisions and products vectorised in float32, the sums in float64."""
+    G, hw, lut = d["G"], np.float32(d["hw"]), d["lut"]
+    ks = np.float32(len(lut) - 1) / hw
+    g = np.zeros((G, G, G, 2))
+    ax = np.arange(G, dtype=np.float32)
+    for s in range(d["n"]):
+        dx = np.abs(ax - d["x"][s]); dy = np.abs(ax - d["y"][s]); dz = np.abs(ax - d["z"][s])
+        mx, my, mz = dx < hw, dy < hw, dz < hw
+        if not (mx.any() and my.any() and mz.any()):
+            continue
+        wx = np.where(mx, lut[np.where(mx, (dx * ks).astype(np.int64), 0)], 0).astype(np.float32)
+        wy = np.where(my, lut[np.where(my, (dy * ks).astype(np.int64), 0)], 0).astype(np.float32)
+        wz = np.where(mz, lut[np.where(mz, (dz * ks).astype(np.int64), 0)], 0).astype(np.float32)
+        w = (wy[:, None] * wx[None, :])[None, :, :] * wz[:, None, None]          # (wx*wy)*wz in fp32
+        g[..., 0] += (w * d["re"][s]).astype(np.float64)
+        g[..., 1] += (w * d["im"][s]).astype(np.float64)
+    return g
+
+
+def test_gridding_matches_numpy_bruteforce():
+    d = synth.preset("gridding", "tiny", n=400, seed=2)
+    assert np.allclose(T().gridding(d), _gridding_numpy(d), rtol=0, atol=1e-12)
+
+
+def test_gridding_single_sample_closed_form():
+    """One sample exactly on grid point (5, 6, 7) with value 1: the grid holds
+    the separable table lut[(int)(|d| ks)]^3 around it, 0 elsewhere."""
+    d = synth.preset("gridding", "tiny", seed=3)
+    one = dict(d, n=1, x=np.array([5.0], np.float32), y=np.array([6.0], np.float32), z=np.array([7.0], np.float32),
+               re=np.array([1.0], np.float32), im=np.array([0.0], np.float32))
+    g = T().gridding(one)
+    lut, hw = d["lut"], d["hw"]
+    ks = np.float32(len(lut) - 1) / np.float32(hw)
+    assert g[7, 6, 5, 0] == 1.0 and not g[..., 1].any()
+    w1 = lut[int(np.float32(1.0) * ks)]
+    assert g[7, 6, 6, 0] == pytest.approx(float(np.float32(np.float32(w1 * lut[0]) * lut[0])), rel=0)
+    assert np.count_nonzero(g[..., 0]) == (2 * int(np.ceil(hw)) - 1) ** 3
+
+
+def test_gridding_is_linear():
+    d = synth.preset("gridding", "tiny", seed=4)
+    h = d["n"] // 2
+    part = lambda sl: dict(d, n=len(d["x"][sl]), **{k: np.ascontiguousarray(d[k][sl]) for k in ("x", "y", "z", "re", "im")})  # noqa: E731
+    a, b = T().gridding(part(slice(0, h))), T().gridding(part(slice(h, None)))
+    assert np.allclose(T().gridding(d), a + b, rtol=0, atol=1e-12)
