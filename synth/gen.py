@@ -271,20 +271,26 @@ def gen_histo_raw(n: int, bins: int, iters: int, seed: int = 0) -> dict:
 
 
 def gen_gridding(G: int, n: int, W: float = 4.0, L: int = 1024, seed: int = 0) -> dict:
-    """MRI k-space samples for gridding [ext Parboil mri-gridding]: n points on
-    a few radial-ish spokes plus uniform jitter inside [0, G)^3 (denser near
-    the centre, like a radial acquisition), complex values U[-1, 1)^2; the
+    """MRI k-space samples for gridding [ext Parboil mri-gridding]: half
+    uniform in [0, G)^3, half on 64 jittered radial spokes (a radial
+    acquisition's lines), complex values U[-1, 1)^2; the
     separable Kaiser-Bessel kernel of width W (half-width W/2) tabulated at L
     points, beta = pi sqrt((W/2)^2 (2 - 0.5)^2 - 0.8) (oversampling 2),
     normalised to 1 at distance 0 -- computed here in fp64."""
     r = rng(seed)
     hw = W / 2.0
     c = G / 2.0
-    t = r.uniform(-1, 1, n) ** 3                      # denser near the centre
+    # half the samples uniform in the volume, half on 64 jittered radial
+    # spokes with radius pdf ~ r^2 (each spoke's samples spread like a ball's
+    # volume: no 1/r^2 pile-up at the centre that would leave one gridding
+    # tile with 50x the average work)
+    nu = n // 2
+    t = np.cbrt(r.uniform(0, 1, n - nu)) * r.choice([-1.0, 1.0], n - nu)
     dirs = r.normal(0, 1, (64, 3))
     dirs /= np.linalg.norm(dirs, axis=1, keepdims=True)
-    pick = dirs[r.integers(0, 64, n)]
-    pts = c + (G / 2.0 - hw) * t[:, None] * pick + r.normal(0, 1.5, (n, 3))
+    pick = dirs[r.integers(0, 64, n - nu)]
+    spokes = c + (G / 2.0 - hw) * t[:, None] * pick + r.normal(0, 1.0, (n - nu, 3))
+    pts = np.concatenate([r.uniform(0, G, (nu, 3)), spokes])
     pts = np.clip(pts, 0.0, np.nextafter(G, 0))
     beta = np.pi * np.sqrt((W / 2.0) ** 2 * (2.0 - 0.5) ** 2 - 0.8)
     dist = np.arange(L) * hw / (L - 1)

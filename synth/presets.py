@@ -68,7 +68,7 @@ PRESETS: dict[str, dict[str, dict]] = {
     "gridding": {
         "tiny": dict(G=24, n=3000),
         "small": dict(G=48, n=40000),
-        "default": dict(G=128, n=1 << 20),
+        "default": dict(G=128, n=1 << 19),
     },
     "lbm": {
         "tiny": dict(nx=20, ny=11, nz=9, steps=3),
