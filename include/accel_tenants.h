@@ -66,6 +66,8 @@ typedef struct {
   float c0, c1;
   const accel_tmap *gmaps;  /* diagnostic: non-NULL = read the three maps from
                                this DEVICE array instead of the parameters */
+  const float *a0;          /* the input volume (kernel "stencil_bulk": 1-D
+                               bulk copies need no tensor map) */
 } accel_stencil_tma_args;
 
 /* histo -- saturating histogram (Parboil histo main + final fused).

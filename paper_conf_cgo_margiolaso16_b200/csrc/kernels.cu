@@ -115,6 +115,7 @@ const Builtin kBuiltins[] = {
     {"stencil_x", &make_desc<StencilX>},
     {"stencil_deep", &make_desc<StencilDeep>},
     {"stencil_tma", &make_desc<StencilTma>},
+    {"stencil_bulk", &make_desc<StencilBulk>},
     {"histo", &make_desc<Histo>},
     {"histo_wide", &make_desc<HistoWide>},
     {"histo_prescan", &make_desc<HistoPrescan>},

@@ -33,7 +33,12 @@
 
 namespace accel {
 
-struct StencilTma {
+// kBulk: the same ring filled by plain 1-D bulk copies (cp.async.bulk, one
+// per in-volume row segment of a plane) instead of 3-D tensor boxes: no
+// tensor map; rows and columns outside the volume are not copied (their smem
+// holds stale values that only feed face cells, which copy the input).
+template <bool kBulk>
+struct StencilTmaT {
   using Args = accel_stencil_tma_args;
   static constexpr int kConsumers = 8;
   static constexpr int kThreads = 32 * (kConsumers + 1);
@@ -89,10 +94,30 @@ struct StencilTma {
         // launch, or -- for a RESOLVE top-up CTA -- by other CTAs of this
         // grid, ordered by the dispatch's wait_complete and the barrier above)
         asm volatile("fence.proxy.async.global;" ::: "memory");
+        // bulk path: the plane's in-volume row segments (16-B aligned: nx % 4 == 0)
+        const int xs = max(x0 - 4, 0), xe = min(x0 + kTX + 4, nx);
+        const uint32_t rowb = 4u * (uint32_t)(xe - xs), dcol = 4u * (uint32_t)(xs - (x0 - 4));
+        const int ys = max(y0 - 1, 0), ye = min(y0 + kTY + 1, ny);
+        const float* in = r == 0 ? a.a0 : ((r & 1u) ? a.buf0 : a.buf1);
         for (int p = 0; p < nplanes; ++p) {
           if (p >= kNS) mbar_wait(empty(p), (uint32_t)((p / kNS) - 1) & 1u);
-          mbar_expect_tx(full(p), kPlaneBytes);
-          tma_load_3d(slot(p), map, x0 - 4, y0 - 1, z0 - 1 + p, full(p));
+          if constexpr (kBulk) {
+            const int z = z0 - 1 + p;
+            if (z < 0 || z >= nz) {
+              mbar_arrive(full(p));   // nothing to copy: a face plane
+              continue;
+            }
+            mbar_expect_tx(full(p), rowb * (uint32_t)(ye - ys));
+            for (int y = ys; y < ye; ++y) {
+              const float* g = in + ((size_t)z * ny + y) * nx + xs;
+              const uint32_t dst = slot(p) + 4u * (uint32_t)((y - (y0 - 1)) * kCols) + dcol;
+              asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];"
+                           ::"r"(dst), "l"(g), "r"(rowb), "r"(full(p)) : "memory");
+            }
+          } else {
+            mbar_expect_tx(full(p), kPlaneBytes);
+            tma_load_3d(slot(p), map, x0 - 4, y0 - 1, z0 - 1 + p, full(p));
+          }
         }
       }
       return;   // (the dispatch loop's barrier follows)
@@ -157,5 +182,8 @@ struct StencilTma {
     }
   }
 };
+
+using StencilTma = StencilTmaT<false>;
+using StencilBulk = StencilTmaT<true>;
 
 }  // namespace accel

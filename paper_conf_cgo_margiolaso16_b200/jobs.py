@@ -194,13 +194,14 @@ class StencilJob(Job):
             ("stencil" if self.nx % 4 == 0 else "stencil_x")
         if kernel != "stencil_x" and self.nx % 4:
             raise ValueError(f"{kernel} needs nx % 4 == 0 (16-B rows); stencil_x takes any nx")
-        if kernel == "stencil_tma":
+        if kernel in ("stencil_tma", "stencil_bulk"):
             # 3-D maps of a0, buf0, buf1: box = one staged plane (136 x 10 x 1)
             maps = b"".join(abi.accel_tma_map_3d(t.data_ptr(), self.nx, self.ny, self.nz, 136, 10, 1)
                             for t in (self.inputs["a0"], self.buf[0], self.buf[1]))
             self.args = abi.accel_stencil_tma_args((C.c_uint8 * 384).from_buffer_copy(maps), self.buf[0].data_ptr(),
                                                    self.buf[1].data_ptr(), self.nx, self.ny, self.nz,
                                                    d["c0"], d["c1"])
+            self.args.a0 = self.inputs["a0"].data_ptr()
             if d.get("tma_global_maps"):   # diagnostic (scripts/diag_tma.py)
                 self.gmaps = torch.frombuffer(bytearray(maps), dtype=torch.uint8).to(self.device)
                 self.args.gmaps = self.gmaps.data_ptr()

@@ -324,6 +324,8 @@ def _stencil_fp32_replica(d):
 
 
 @pytest.mark.parametrize("kernel,over", [("stencil_tma", dict(nx=136, ny=17, nz=19, sweeps=4)),
+                                         ("stencil_bulk", dict(nx=136, ny=17, nz=19, sweeps=4)),
+                                         ("stencil_bulk", dict(nx=260, ny=9, nz=8, sweeps=3)),
                                          ("stencil", dict(nx=136, ny=17, nz=19, sweeps=4)),
                                          ("stencil_x", dict(nx=70, ny=21, nz=19, sweeps=3))])
 def test_stencil_bit_exact_fp32_sequence(acc_tiny_caps, kernel, over):
