@@ -64,6 +64,8 @@ typedef struct {
   float *buf1;
   uint32_t nx, ny, nz;
   float c0, c1;
+  uint32_t l2hint;          /* diagnostic: 1 = tensor loads with an L2
+                               evict_first cache policy, 2 = evict_last */
   const accel_tmap *gmaps;  /* diagnostic: non-NULL = read the three maps from
                                this DEVICE array instead of the parameters */
   const float *a0;          /* the input volume (kernel "stencil_bulk": 1-D

@@ -116,7 +116,11 @@ struct StencilTmaT {
             }
           } else {
             mbar_expect_tx(full(p), kPlaneBytes);
-            tma_load_3d(slot(p), map, x0 - 4, y0 - 1, z0 - 1 + p, full(p));
+            if (a.l2hint == 0)
+              tma_load_3d(slot(p), map, x0 - 4, y0 - 1, z0 - 1 + p, full(p));
+            else
+              tma_load_3d_hint(slot(p), map, x0 - 4, y0 - 1, z0 - 1 + p, full(p),
+                               a.l2hint == 1 ? policy_evict_first() : policy_evict_last());
           }
         }
       }

@@ -202,6 +202,7 @@ class StencilJob(Job):
                                                    self.buf[1].data_ptr(), self.nx, self.ny, self.nz,
                                                    d["c0"], d["c1"])
             self.args.a0 = self.inputs["a0"].data_ptr()
+            self.args.l2hint = int(d.get("l2hint", os.environ.get("ACCEL_TMA_L2HINT", 0)))
             if d.get("tma_global_maps"):   # diagnostic (scripts/diag_tma.py)
                 self.gmaps = torch.frombuffer(bytearray(maps), dtype=torch.uint8).to(self.device)
                 self.args.gmaps = self.gmaps.data_ptr()
