@@ -109,6 +109,31 @@ struct Cutcp {
     auto clampc = [&](int v) { return v < 0 ? 0 : (v >= nc ? nc - 1 : v); };
     const int cy0 = clampc((int)floorf((by0 - cm) / cs)), cy1 = clampc((int)floorf((by1 + cm) / cs));
     const int cz0 = clampc((int)floorf((bz0 - cm) / cs)), cz1 = clampc((int)floorf((bz1 + cm) / cs));
+    // the cell rows' trimmed atom ranges are packed back to back into the
+    // shared tile (a row of 2-A cells holds a few atoms), which is evaluated
+    // whenever it is full: two barriers per 128 atoms instead of per row
+    auto evaluate = [&](int n) {
+#pragma unroll 2
+      for (int q = 0; q < n; ++q) {
+        const float4 at = tile[q];
+        const float dx = __fsub_rn(px, at.x), dy = __fsub_rn(py, at.y);
+        const float dxy = __fadd_rn(__fmul_rn(dx, dx), __fmul_rn(dy, dy));
+#pragma unroll
+        for (int p = 0; p < kPts; ++p) {
+          const float dz = __fsub_rn(pz[p], at.z);
+          const float r2 = __fadd_rn(dxy, __fmul_rn(dz, dz));
+          r2min[p] = fminf(r2min[p], r2);
+          if (r2 < c2) {
+            // explicit FMAs: the same op sequence in every instantiation
+            // (native and persistent must agree bit for bit)
+            const float s = __fmaf_rn(-r2, inv_c2, 1.0f);
+            const float qs = __fmul_rn(__fmul_rn(at.w, rsqrt_ftz(r2)), s);
+            sum[p] = __fmaf_rn(qs, s, sum[p]);
+          }
+        }
+      }
+    };
+    int fill = 0;   // atoms staged in the tile (uniform)
     for (int cz = cz0; cz <= cz1; ++cz) {
       const float gz = gap(bz0, bz1, cz * cs, (cz + 1) * cs);
       for (int cy = cy0; cy <= cy1; ++cy) {
@@ -118,31 +143,27 @@ struct Cutcp {
         const float rx = sqrtf(cm * cm - d2);
         const int cx0 = clampc((int)floorf((bx0 - rx) / cs)), cx1 = clampc((int)floorf((bx1 + rx) / cs));
         const int row = (cz * nc + cy) * nc;
-        const int a0 = __ldg(a.cell_start + row + cx0), a1 = __ldg(a.cell_start + row + cx1 + 1);
-        for (int base = a0; base < a1; base += kTile) {
-          const int n = min(kTile, a1 - base);
-          __syncthreads();
-          if (t < n) tile[t] = __ldg(reinterpret_cast<const float4*>(a.atoms) + base + t);
-          __syncthreads();
-#pragma unroll 2
-          for (int q = 0; q < n; ++q) {
-            const float4 at = tile[q];
-            const float dx = __fsub_rn(px, at.x), dy = __fsub_rn(py, at.y);
-            const float dxy = __fadd_rn(__fmul_rn(dx, dx), __fmul_rn(dy, dy));
-#pragma unroll
-            for (int p = 0; p < kPts; ++p) {
-              const float dz = __fsub_rn(pz[p], at.z);
-              const float r2 = __fadd_rn(dxy, __fmul_rn(dz, dz));
-              r2min[p] = fminf(r2min[p], r2);
-              if (r2 < c2) {
-                const float s = 1.0f - r2 * inv_c2;
-                sum[p] += at.w * rsqrt_ftz(r2) * s * s;
-              }
-            }
+        int a0 = __ldg(a.cell_start + row + cx0);
+        const int a1 = __ldg(a.cell_start + row + cx1 + 1);
+        while (a0 < a1) {
+          const int take = min(kTile - fill, a1 - a0);
+          if (t < take) tile[fill + t] = __ldg(reinterpret_cast<const float4*>(a.atoms) + a0 + t);
+          fill += take;
+          a0 += take;
+          if (fill == kTile) {
+            __syncthreads();
+            evaluate(kTile);
+            __syncthreads();
+            fill = 0;
           }
         }
       }
     }
+    if (fill) {
+      __syncthreads();
+      evaluate(fill);
+    }
+    __syncthreads();   // the CTA's next VG reuses the tile
     if (i < (int)a.nx && j < (int)a.ny) {
 #pragma unroll
       for (int p = 0; p < kPts; ++p) {
