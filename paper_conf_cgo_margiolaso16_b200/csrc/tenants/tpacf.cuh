@@ -21,6 +21,9 @@
 #ifndef TPACF_UNROLL2
 #define TPACF_UNROLL2 1
 #endif
+#ifndef TPACF_LUT
+#define TPACF_LUT 1
+#endif
 
 namespace accel {
 
@@ -35,8 +38,10 @@ struct Tpacf {
   static constexpr int kTile = 256;
   // [warp][bin][lane] u32 counters + Q tile (256 float4: x, y, z, pad; one
   // LDS.128 per pair) + edges (32)
-  static constexpr uint32_t kDynSmem =
-      kWarps * kMaxBins * 32 * sizeof(uint32_t) + kTile * sizeof(float4) + 32 * sizeof(float);
+  // + the exponent table (30 float4, below; 6 CTAs/SM still fit)
+  static constexpr int kLut = 30;
+  static constexpr uint32_t kDynSmem = kWarps * kMaxBins * 32 * sizeof(uint32_t) + kTile * sizeof(float4) +
+                                       32 * sizeof(float) + kLut * sizeof(float4);
 
   // Dequeue-order cost model (dispatch.cuh accel_lpt_order): Q tiles the VG
   // walks -- DD / RR blocks (y <= S) start at their diagonal tile, DR blocks
@@ -92,6 +97,39 @@ struct Tpacf {
                 iz = have ? __ldg(P + 2 * n + i) : 0.f;
     uint32_t* myh = hist + warp * kMaxBins * 32 + lane;
     __syncthreads();   // edges staged
+    // Exponent table (exact): u = 1 - d in fp32 is monotone in d, so the
+    // (clamped) exponent field of u orders d against every edge whose
+    // u-exponent cell differs; only the (at most two) edges sharing d's cell
+    // need a compare.  Cell c in 0..28 = exponent field min(max(e, 102), 130)
+    // - 102 (u = 0, i.e. d = 1, and u < 2^-24 fall in cell 0; fp32 d has no
+    // value strictly between), cell 29 = u < 0 (d > 1).  Entry c = (edges in
+    // lower cells -- all greater than d --, candidate 1, candidate 2).  The
+    // bins are log-spaced in angle, so consecutive edges are more than an
+    // octave apart in u; an input with three edges in one cell falls back to
+    // the binary search.
+    float4* lut = reinterpret_cast<float4*>(edges + 32);
+    auto cell_of = [](uint32_t ub) {
+      return (ub >> 31) ? kLut - 1 : min(max((int)(ub >> 23), 102), 130) - 102;
+    };
+    bool crowded = false;
+    if (TPACF_LUT && t < kLut) {
+      int base = 0, nc = 0;
+      float c1 = -3.0f, c2 = -3.0f;
+      for (uint32_t k = 0; k < ne; ++k) {
+        const float e = edges[k];
+        const int ce = cell_of(__float_as_uint(__fsub_rn(1.0f, e)));
+        // an edge above 1 (cell 29) exceeds every d <= 1
+        const bool lower = t < kLut - 1 && (ce < t || ce == kLut - 1);
+        if (lower) ++base;
+        if (ce == t) {
+          if (nc == 0) c1 = e; else c2 = e;
+          ++nc;
+        }
+      }
+      crowded = nc > 2;
+      lut[t] = make_float4(__int_as_float(base), c1, c2, 0.f);
+    }
+    const bool use_lut = TPACF_LUT && !__syncthreads_or(crowded);
     const float e7 = edges[7], e15 = edges[15], e23 = edges[23];
     uint32_t tile0, tile1;
     tile_range(a, vb, tile0, tile1);
@@ -104,9 +142,14 @@ struct Tpacf {
       const uint32_t cnt = min((uint32_t)kTile, n - jt);
       // pairs i < j on the diagonal tile start after i
       const uint32_t q0 = (upper && jt == vb.x * kTile) ? (uint32_t)t + 1 : 0u;
-      // bin = #{k : d < edges[k]}; edges descending -> binary search, its
-      // first two levels from registers (edges[15], then edges[7] / [23])
-      auto bin_of = [&](float d) {
+      // bin = #{k : d < edges[k]}: the exponent table, else a binary search
+      // over the descending edges, its first two levels from registers
+      // (edges[15], then edges[7] / [23])
+      auto bin_lut = [&](float d) {
+        const float4 L = lut[cell_of(__float_as_uint(__fsub_rn(1.0f, d)))];
+        return __float_as_int(L.x) + (d < L.y ? 1 : 0) + (d < L.z ? 1 : 0);
+      };
+      auto bin_search = [&](float d) {
         int m = (e15 > d) ? 16 : 0;
         if (((m != 0) ? e23 : e7) > d) m += 8;
 #pragma unroll
@@ -127,16 +170,25 @@ struct Tpacf {
 #endif
       };
       uint32_t q = q0;
+      if (use_lut) {
+        for (; q + 1 < cnt; q += 2) {
+          const int m0 = bin_lut(dot(qt[q])), m1 = bin_lut(dot(qt[q + 1]));
+          count(m0);
+          count(m1);
+        }
+        for (; q < cnt; ++q) count(bin_lut(dot(qt[q])));
+      } else {
 #if TPACF_UNROLL2
-      // two independent search chains in flight (their shared-memory edge
-      // loads overlap)
-      for (; q + 1 < cnt; q += 2) {
-        const int m0 = bin_of(dot(qt[q])), m1 = bin_of(dot(qt[q + 1]));
-        count(m0);
-        count(m1);
-      }
+        // two independent search chains in flight (their shared-memory edge
+        // loads overlap)
+        for (; q + 1 < cnt; q += 2) {
+          const int m0 = bin_search(dot(qt[q])), m1 = bin_search(dot(qt[q + 1]));
+          count(m0);
+          count(m1);
+        }
 #endif
-      for (; q < cnt; ++q) count(bin_of(dot(qt[q])));
+        for (; q < cnt; ++q) count(bin_search(dot(qt[q])));
+      }
     }
     __syncthreads();
     if (t < (int)ne + 1) {

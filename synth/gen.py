@@ -92,7 +92,7 @@ def gen_bfs(nv: int, deg_lo: int = 1, deg_hi: int = 11, src: int = 0, seed: int 
 
 
 def gen_cutcp(box: float, density: float = 0.1, h: float = 0.5, cutoff: float = 12.0,
-              excl: float = 1.0, cell: float = 2.0, seed: int = 0) -> dict:
+              excl: float = 1.0, cell: float = 4.0, seed: int = 0) -> dict:
     """Water-like charges in a cubic box [0, box)^3.
 
     Molecules = O(-0.834) at a uniform position plus two H(+0.417) at a ~1 A

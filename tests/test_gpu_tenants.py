@@ -371,3 +371,21 @@ def test_histo_pipeline_default(acc, oracle_lib):
     nat, sh, _ = run_modes(acc, lambda: HistoPipelineJob(d))
     for r in (nat, sh):
         assert (r["lo"], r["hi"]) == (lo, hi) and np.array_equal(r["counts"], counts)
+
+
+@pytest.mark.parametrize("edges", ["linear", "near_one"])
+def test_tpacf_custom_edges(acc_tiny_caps, oracle_lib, edges):
+    """Bin edges the exponent table cannot separate (many edges in one octave
+    of 1 - d: the binary-search fallback) and edges crowding d = 1: still
+    bit-exact against the oracle."""
+    from paper_conf_cgo_margiolaso16_b200.jobs import TpacfJob
+    d = synth.preset("tpacf", "tiny", seed=12)
+    if edges == "linear":
+        b = np.linspace(0.99, -0.9, 21)
+    else:
+        b = 1.0 - np.geomspace(1e-7, 1.5, 21)
+    d = dict(d, binb=np.ascontiguousarray(np.sort(b)[::-1].astype(np.float32)))
+    nat, sh, _ = run_modes(acc_tiny_caps, lambda: TpacfJob(d))
+    dd, rr, dr = oracle_lib.tpacf(d)
+    for r in (nat, sh):
+        assert np.array_equal(r["dd"], dd) and np.array_equal(r["rr"], rr) and np.array_equal(r["dr"], dr)
