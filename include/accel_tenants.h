@@ -206,6 +206,14 @@ typedef struct {
   uint32_t m, n, k;
 } accel_sgemm_tc_args;
 
+/* sgemm_tc1 -- the same product in one step: tmaps = DEVICE pointer to TWO
+ * CUtensorMaps over the raw fp32 operands (A [m][k], box 16 x 128; B [n][k],
+ * box 16 x 256; 64-B swizzle; row stride 4k bytes, so k % 4 == 0 -- TMA needs
+ * 16-B aligned rows).  Each CTA splits every landed 32-wide slab into hi/lo in
+ * shared memory before the MMAs; no hi/lo arrays in global memory.  Same
+ * block, VG and grid as sgemm_tc; the k % 4 != 0 case takes split + tc. */
+typedef accel_sgemm_tc_args accel_sgemm_tc1_args;
+
 /* sad -- Parboil "sad" (H.264 motion estimation), three
  * kernels sharing one argument struct, run as the three steps of a request:
  *   "sad_4x4"   sad4[mb][p][b] = sum over the 4x4 sub-block b of the 16x16

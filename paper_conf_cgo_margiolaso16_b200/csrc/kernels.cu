@@ -127,6 +127,7 @@ const Builtin kBuiltins[] = {
     {"sgemm", &make_desc<Sgemm>},
     {"sgemm_split", &make_desc<SgemmSplit>},
     {"sgemm_tc", &make_desc<SgemmTc>},
+    {"sgemm_tc1", &make_desc<SgemmTc1>},
     {"lbm", &make_desc<Lbm>},
     {"gridding_binning", &make_desc<GridBinning>},
     {"gridding_scan_l1", &make_desc<GridScanL1>},

@@ -270,3 +270,227 @@ struct SgemmTc {
 };
 
 }  // namespace accel
+
+namespace accel {
+
+// sgemm_tc1 -- the same 3xTF32 tensor-core GEMM in ONE step:
+// TMA loads the fp32 A and B tiles as they are; the 16 accumulator warps,
+// idle between accumulator hand-overs, split every landed slab in place and
+// release it to the MMA issuer.  No split launch, no hi/lo operand arrays in
+// HBM (4 x 64 MB at 4096^3), one launch per request.  Rows must be 16-B
+// aligned for TMA (k % 4 == 0); other k keep the two-step path.
+//
+//  * hi = x truncated to TF32.  kind::tf32 reads the fp32 word and ignores its
+//    low 13 mantissa bits, so the raw tile already IS A_hi / B_hi and only
+//    lo = x - hi is written (to a second buffer at the same swizzled offsets:
+//    the split is elementwise, the layout is unchanged).  Truncation leaves
+//    |lo| < 2^-10 |x| (vs 2^-11 for a round-to-nearest hi), still far inside
+//    the 3xTF32 error bound the parity tests hold.
+//  * Slabs are 16 wide (64-B rows, SWIZZLE_64B) so that FOUR stages of
+//    raw+lo (48 KB each) fit: a slab's conversion waits for the MMA four slabs
+//    back, not two (with 32-wide slabs only two 96-KB stages fit and the
+//    tensor pipe idled through every TMA + conversion).
+//  * The converters read accumulator group h out of TMEM only after they
+//    converted the first slab of group h+2 -- by then group h's MMAs are long
+//    done, so the hand-over never stalls a conversion, while the MMAs of
+//    group h+1 keep the tensor pipe busy.
+#ifndef SGEMM1_TRUNC
+#define SGEMM1_TRUNC 1
+#endif
+
+__device__ __forceinline__ uint64_t umma_desc_k_sw64(uint32_t saddr) {
+  // K-major, 64-B swizzle: rows of 64 B, 8-row groups 512 B apart (SBO),
+  // version 1 (sm_100), layout type 4 = SWIZZLE_64B
+  return (uint64_t)((saddr >> 4) & 0x3FFFu) | ((uint64_t)1u << 16) | ((uint64_t)(512u >> 4) << 32) |
+         ((uint64_t)1u << 46) | ((uint64_t)4u << 61);
+}
+
+struct SgemmTc1 {
+  using Args = accel_sgemm_tc_args;   // tmaps: A, B (raw fp32, box 16 x 128 / 16 x 256, SWIZZLE_64B)
+  static constexpr int kThreads = 640;
+  static constexpr int kAccWarp0 = 4, kAccWarps = 16;
+  static constexpr uint32_t kChunk = 1;
+  static constexpr int kMinBlocks = 1;
+  static constexpr int kBM = 128, kBN = 256, kBK = 16;
+  static constexpr int kStages = 4;
+#ifndef SGEMM1_GROUP
+#define SGEMM1_GROUP 4
+#endif
+  static constexpr int kGroup = SGEMM1_GROUP;             // slabs per accumulator hand-over (64 k)
+  static constexpr uint32_t kTileA = kBM * kBK * 4;      // 8 KB
+  static constexpr uint32_t kTileB = kBN * kBK * 4;      // 16 KB
+  // per stage: A (raw = hi), A_lo, B (raw = hi), B_lo
+  static constexpr uint32_t kStage = 2 * kTileA + 2 * kTileB;   // 48 KB
+  static constexpr uint32_t kTmemCols = 512;
+  static constexpr uint32_t kDynSmem = kStages * kStage + 1024 + 1024;
+  static constexpr uint32_t kIdesc = SgemmTc::kIdesc;
+  static constexpr int kF4 = (int)(kTileA + kTileB) / 16 / 512;   // float4 per converter thread per slab
+
+  static __device__ __forceinline__ float trunc_tf32(float x) { return __uint_as_float(__float_as_uint(x) & 0xFFFFE000u); }
+
+  static __device__ __forceinline__ void body(const Args& a, const VirtualBlock& vb, char* smem_raw) {
+    using namespace tc;
+    const uint32_t warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    char* smem = reinterpret_cast<char*>((reinterpret_cast<uintptr_t>(smem_raw) + 1023) & ~uintptr_t(1023));
+    const uint32_t sbase = smem_u32(smem);
+    // barriers: full[S], empty[S], conv[S], accfull[2], accempty[2]
+    const uint32_t bars = sbase + kStages * kStage;
+    auto full = [&](int s) { return bars + 8u * s; };
+    auto empty = [&](int s) { return bars + 8u * (kStages + s); };
+    auto conv = [&](int s) { return bars + 8u * (2 * kStages + s); };
+    auto accfull = [&](int b) { return bars + 8u * (3 * kStages + b); };
+    auto accempty = [&](int b) { return bars + 8u * (3 * kStages + 2 + b); };
+    uint32_t* tmem_slot = reinterpret_cast<uint32_t*>(smem + kStages * kStage + 256);
+    const CUtensorMap* maps = reinterpret_cast<const CUtensorMap*>(a.tmaps);
+    const int m0 = (int)vb.y * kBM, n0 = (int)vb.x * kBN;
+    const int nk = ((int)a.k + kBK - 1) / kBK;
+    const int ng = (nk + kGroup - 1) / kGroup;
+    // stage s: A at +0, A_lo at +kTileA, B at +2 kTileA, B_lo at +2 kTileA + kTileB
+    auto st = [&](int s) { return sbase + (uint32_t)s * kStage; };
+
+    if (threadIdx.x == 0) {
+      for (int s = 0; s < kStages; ++s) {
+        mbar_init(full(s), 1);
+        mbar_init(empty(s), 1);
+        mbar_init(conv(s), kAccWarps);
+      }
+      for (int b = 0; b < 2; ++b) {
+        mbar_init(accfull(b), 1);
+        mbar_init(accempty(b), kAccWarps);
+      }
+      asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+      asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+    }
+    if (warp == 2) {
+      asm volatile("tcgen05.alloc.cta_group::1.sync.aligned.shared::cta.b32 [%0], %1;" ::"r"(smem_u32(tmem_slot)),
+                   "r"(kTmemCols)
+                   : "memory");
+    }
+    fence_before();
+    __syncthreads();
+    fence_after();
+    const uint32_t tmem = *tmem_slot;
+
+    if (warp == 0 && lane == 0) {
+      // ---- TMA producer: raw fp32 slabs of A and B
+      tmap_acquire(&maps[0]);
+      tmap_acquire(&maps[1]);
+      for (int kb = 0; kb < nk; ++kb) {
+        const int s = kb % kStages;
+        if (kb >= kStages) mbar_wait(empty(s), ((kb / kStages) - 1) & 1);
+        mbar_expect_tx(full(s), kTileA + kTileB);
+        tma_load_2d(st(s), &maps[0], kb * kBK, m0, full(s));
+        tma_load_2d(st(s) + 2 * kTileA, &maps[1], kb * kBK, n0, full(s));
+      }
+    } else if (warp == 1 && lane == 0) {
+      // ---- MMA issuer: waits for the converted slab (conv), not for TMA
+      for (int g = 0; g < ng; ++g) {
+        const int b = g & 1;
+        if (g >= 2) mbar_wait(accempty(b), ((g >> 1) - 1) & 1);
+        fence_after();
+        const uint32_t dacc = tmem + (uint32_t)(b * kBN);
+        const int kb1 = min(nk, (g + 1) * kGroup);
+        for (int kb = g * kGroup; kb < kb1; ++kb) {
+          const int s = kb % kStages;
+          mbar_wait(conv(s), (kb / kStages) & 1);
+          fence_after();
+          const uint32_t sa = st(s);
+#pragma unroll
+          for (int ks = 0; ks < kBK / 8; ++ks) {
+            const uint32_t koff = ks * 32;   // 8 tf32 = 32 B along the 64-B swizzled row
+            const uint64_t ahi = umma_desc_k_sw64(sa + koff);
+            const uint64_t alo = umma_desc_k_sw64(sa + kTileA + koff);
+            const uint64_t bhi = umma_desc_k_sw64(sa + 2 * kTileA + koff);
+            const uint64_t blo = umma_desc_k_sw64(sa + 2 * kTileA + kTileB + koff);
+            mma_tf32(dacc, ahi, bhi, kIdesc, (kb != g * kGroup || ks != 0) ? 1u : 0u);
+            mma_tf32(dacc, ahi, blo, kIdesc, 1u);
+            mma_tf32(dacc, alo, bhi, kIdesc, 1u);
+          }
+          // the last kStages slabs are never refilled: no arrival outlives the VG
+          if (kb + kStages < nk) mma_commit(empty(s));
+        }
+        mma_commit(accfull(b));
+      }
+    } else if (warp >= (uint32_t)kAccWarp0) {
+      // ---- converters + accumulators
+      const uint32_t q = warp & 3u, h = (warp - kAccWarp0) >> 2;
+      const uint32_t ct = threadIdx.x - 32u * kAccWarp0;   // 0..511
+      float acc[64];
+#pragma unroll
+      for (int j = 0; j < 64; ++j) acc[j] = 0.f;
+      auto split_slab = [&](int kb) {
+        const int s = kb % kStages;
+        mbar_wait(full(s), (kb / kStages) & 1);
+        const uint32_t sa = st(s);
+        constexpr uint32_t kA4 = kTileA / 16;   // float4 of A; then those of B
+        float4 xs[kF4];
+#pragma unroll
+        for (int i = 0; i < kF4; ++i) {   // all loads in flight before the first store
+          const uint32_t f = ct + 512u * (uint32_t)i;
+          xs[i] = lds_f4(f < kA4 ? sa + 16u * f : sa + 2 * kTileA + 16u * (f - kA4));
+        }
+#pragma unroll
+        for (int i = 0; i < kF4; ++i) {
+          const uint32_t f = ct + 512u * (uint32_t)i;
+          const uint32_t raw = f < kA4 ? sa + 16u * f : sa + 2 * kTileA + 16u * (f - kA4);
+          const uint32_t lo = f < kA4 ? raw + kTileA : raw + kTileB;
+          const float4 x = xs[i];
+#if SGEMM1_TRUNC
+          const float4 hi = make_float4(trunc_tf32(x.x), trunc_tf32(x.y), trunc_tf32(x.z), trunc_tf32(x.w));
+#else
+          const float4 hi = make_float4(SgemmSplit::hi_of(x.x), SgemmSplit::hi_of(x.y), SgemmSplit::hi_of(x.z),
+                                        SgemmSplit::hi_of(x.w));
+          asm volatile("st.shared.v4.f32 [%0], {%1, %2, %3, %4};" ::"r"(raw), "f"(hi.x), "f"(hi.y), "f"(hi.z),
+                       "f"(hi.w)
+                       : "memory");
+#endif
+          asm volatile("st.shared.v4.f32 [%0], {%1, %2, %3, %4};" ::"r"(lo), "f"(x.x - hi.x), "f"(x.y - hi.y),
+                       "f"(x.z - hi.z), "f"(x.w - hi.w)
+                       : "memory");
+        }
+        // generic-proxy writes -> read by the tensor cores (async proxy)
+        asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+        __syncwarp();
+        if (lane == 0) mbar_arrive(conv(s));
+      };
+      auto accumulate = [&](int g) {
+        const int b = g & 1;
+        mbar_wait(accfull(b), (g >> 1) & 1);
+        fence_after();
+        const uint32_t taddr = tmem + ((q * 32u) << 16) + (uint32_t)(b * kBN) + h * 64u;
+#pragma unroll
+        for (int c = 0; c < 4; ++c) SgemmTc::ld16_add(taddr + 16u * c, acc + 16 * c);
+        fence_before();
+        __syncwarp();
+        if (lane == 0) mbar_arrive(accempty(b));
+      };
+      int next_acc = 0;
+      for (int kb = 0; kb < nk; ++kb) {
+        split_slab(kb);
+        if (kb % kGroup == 0 && kb / kGroup >= 2) accumulate(next_acc++);
+      }
+      while (next_acc < ng) accumulate(next_acc++);
+      const int row = m0 + (int)(q * 32 + lane);
+      const int c0 = n0 + (int)(h * 64);
+      if (row < (int)a.m) {
+        float* crow = a.c + (size_t)row * a.n;
+        if (c0 + 63 < (int)a.n && (a.n & 3) == 0) {
+#pragma unroll
+          for (int j = 0; j < 64; j += 4)
+            *reinterpret_cast<float4*>(crow + c0 + j) = make_float4(acc[j], acc[j + 1], acc[j + 2], acc[j + 3]);
+        } else {
+#pragma unroll
+          for (int j = 0; j < 64; ++j)
+            if (c0 + j < (int)a.n) crow[c0 + j] = acc[j];
+        }
+      }
+    }
+    fence_before();
+    __syncthreads();
+    fence_after();
+    if (warp == 2)
+      asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, %1;" ::"r"(tmem), "r"(kTmemCols) : "memory");
+  }
+};
+
+}  // namespace accel

@@ -409,13 +409,31 @@ class SgemmJob(Job):
 
 
 class SgemmTcJob(Job):
-    """sgemm on the tcgen05 tensor cores (3xTF32): steps split(A and B), tc."""
+    """sgemm on the tcgen05 tensor cores (3xTF32).  k % 4 == 0 (16-B aligned
+    rows for TMA): one step, sgemm_tc1, splitting hi/lo in shared memory;
+    otherwise two steps, split(A and B) into padded hi/lo arrays, then tc.
+    The one-step form is the default; one_step=False or
+    ACCEL_SGEMM_ONESTEP=0 selects split + tc."""
 
-    def __init__(self, d: dict, device="cuda"):
+    def __init__(self, d: dict, device="cuda", one_step=None):
         super().__init__(name="sgemm", device=torch.device(device))
         self.m, self.n, self.k = d["m"], d["n"], d["k"]
         self.inputs = {"a": _dev(d["a"].ravel(), self.device), "b": _dev(d["b"].ravel(), self.device)}
         m, n, k = self.m, self.n, self.k
+        if one_step is None:
+            one_step = os.environ.get("ACCEL_SGEMM_ONESTEP", "1") != "0"
+        self.one_step = bool(one_step) and k % 4 == 0
+        self.c = torch.empty(m * n, dtype=torch.float32, device=self.device)
+        self.out = {"c": self.c}
+        if self.one_step:
+            maps = b"".join([
+                abi.accel_tma_map_2d(self.inputs["a"].data_ptr(), k, m, 4 * k, 16, 128, swizzle=64),
+                abi.accel_tma_map_2d(self.inputs["b"].data_ptr(), k, n, 4 * k, 16, 256, swizzle=64)])
+            self.tmaps = torch.frombuffer(bytearray(maps), dtype=torch.uint8).to(self.device)
+            self.args_tc = abi.accel_sgemm_tc_args(self.tmaps.data_ptr(), self.c.data_ptr(), m, n, k)
+            self.main_step = 0
+            self.steps = [Step("sgemm_tc1", (_cdiv(n, 256), _cdiv(m, 128), 1), self.args_tc, 1)]
+            return
         kp = _cdiv(k, 4) * 4   # hi/lo row stride: 16-B aligned rows for TMA
         self.split = {x: torch.empty(sz, dtype=torch.float32, device=self.device)
                       for x, sz in (("a_hi", m * kp), ("a_lo", m * kp), ("b_hi", n * kp), ("b_lo", n * kp))}
@@ -425,8 +443,6 @@ class SgemmTcJob(Job):
             abi.accel_tma_map_2d(self.split["b_hi"].data_ptr(), k, n, 4 * kp, 32, 256),
             abi.accel_tma_map_2d(self.split["b_lo"].data_ptr(), k, n, 4 * kp, 32, 256)])
         self.tmaps = torch.frombuffer(bytearray(maps), dtype=torch.uint8).to(self.device)
-        self.c = torch.empty(m * n, dtype=torch.float32, device=self.device)
-        self.out = {"c": self.c}
         s = self.split
         # one launch splits both operands (VGs of A first, then of B)
         self.args_s = abi.accel_sgemm_split_args(self.inputs["a"].data_ptr(), s["a_hi"].data_ptr(),
@@ -444,8 +460,8 @@ class SgemmTcJob(Job):
     def work(self):
         f = 2.0 * self.m * self.n * self.k
         # roofline of the dominant (tc) launch: 3 tf32 products per algorithmic MAC
-        return {"flops": f, "flops_per_launch": f, "bound": "tensor", "launches": 2, "skip_launches": 1,
-                "mma_flops": 3 * f, "peak_tflops": TF32_TENSOR_TFLOPS}
+        return {"flops": f, "flops_per_launch": f, "bound": "tensor", "launches": len(self.steps),
+                "skip_launches": len(self.steps) - 1, "mma_flops": 3 * f, "peak_tflops": TF32_TENSOR_TFLOPS}
 
 
 class MriqJob(Job):

@@ -13,19 +13,26 @@ pytestmark = pytest.mark.gpu
                                        ("small", {}), ("tiny", dict(m=129, n=257, k=36)),
                                        ("tiny", dict(m=130, n=140, k=70)),     # k % 4 == 2: padded hi/lo rows
                                        ("tiny", dict(m=64, n=33, k=33)),       # k % 4 == 1, k not a slab multiple
-                                       ("tiny", dict(m=5, n=7, k=3))])
-def test_sgemm_tc(acc_tiny_caps, oracle_lib, size, over):
+                                       ("tiny", dict(m=5, n=7, k=3)),
+                                       ("tiny", dict(m=300, n=600, k=100)),    # k % 32 == 4: one-step ragged slab
+                                       ("tiny", dict(m=7, n=9, k=4))])
+@pytest.mark.parametrize("one_step", [True, False], ids=["onestep", "twostep"])
+def test_sgemm_tc(acc_tiny_caps, oracle_lib, size, over, one_step):
     from paper_conf_cgo_margiolaso16_b200.jobs import SgemmTcJob
     d = synth.preset("sgemm", size, **over)
-    nat, sh, _ = run_modes(acc_tiny_caps, lambda: SgemmTcJob(d))
+    made = []
+    nat, sh, _ = run_modes(acc_tiny_caps, lambda: made.append(SgemmTcJob(d, one_step=one_step)) or made[-1])
+    assert made[-1].one_step == (one_step and d["k"] % 4 == 0)
     same(nat, sh)
     assert_close_fp32(sh["c"], oracle_lib.sgemm(d), what="sgemm_tc")
 
 
-def test_sgemm_tc_default_sampled(acc, oracle_lib):
+@pytest.mark.parametrize("one_step", [True, False], ids=["onestep", "twostep"])
+def test_sgemm_tc_default_sampled(acc, oracle_lib, one_step):
     from paper_conf_cgo_margiolaso16_b200.jobs import SgemmTcJob
     d = synth.preset("sgemm", "default")
-    job = SgemmTcJob(d)
+    job = SgemmTcJob(d, one_step=one_step)
+    assert job.one_step == one_step and len(job.steps) == (1 if one_step else 2)
     acc.run([job])
     c = job.result()["c"]
     r = np.random.Generator(np.random.PCG64(3))
