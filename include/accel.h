@@ -114,6 +114,14 @@ typedef struct {
   const void *order_fn;       /* host stub of accel_lpt_order<T>: the kernel's
                                  dequeue-order cost model (T::vg_cost); NULL =
                                  none (linear dequeue order)                    */
+  uint32_t max_ctas_per_sm;   /* useful occupancy (T::kMaxCtasPerSm): the kernel
+                                 gains nothing from more resident CTAs per SM
+                                 (measured, scripts/occ_scaling.py), so the
+                                 solver never gives it more than this x SMs --
+                                 the paper's greedy fill "until resource
+                                 saturation" stops at
+                                 the kernel's own saturation and the rest goes
+                                 to its co-runners.  0 = no cap.  SHARED only. */
 } accel_kernel_desc;
 
 /* Fill *out with a built-in tenant kernel: "mop", "stencil", "histo", "bfs",

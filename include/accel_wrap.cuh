@@ -67,6 +67,7 @@ inline int wrap_register(const void* original_fn, const char* name) {
   d.regs = 0;
   d.chunk = T::kChunk;
   d.args_size = sizeof(typename T::Args);
+  d.max_ctas_per_sm = max_ctas_per_sm<T>::value;
   if constexpr (has_vg_cost<T>::value)
     d.order_fn = reinterpret_cast<const void*>(&accel_lpt_order<T>);
   else

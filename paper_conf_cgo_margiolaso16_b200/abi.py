@@ -51,7 +51,8 @@ class accel_kernel_desc(C.Structure):
     _fields_ = [("name", C.c_char_p), ("persistent_fn", vp), ("persistent_resolve_fn", vp), ("native_fn", vp),
                 ("topup_fn", vp),
                 ("block", accel_dim3),
-                ("dyn_smem", u32), ("regs", i32), ("chunk", u32), ("args_size", u32), ("order_fn", vp)]
+                ("dyn_smem", u32), ("regs", i32), ("chunk", u32), ("args_size", u32), ("order_fn", vp),
+                ("max_ctas_per_sm", u32)]
 
 
 class accel_kernel_info(C.Structure):

@@ -188,6 +188,14 @@ struct min_blocks : std::integral_constant<int, 1> {};
 template <class T>
 struct min_blocks<T, std::void_t<decltype(T::kMinBlocks)>> : std::integral_constant<int, T::kMinBlocks> {};
 
+// Optional T::kMaxCtasPerSm: the kernel's useful occupancy (accel_kernel_desc
+// max_ctas_per_sm); 0 = none.
+template <class T, class = void>
+struct max_ctas_per_sm : std::integral_constant<uint32_t, 0> {};
+template <class T>
+struct max_ctas_per_sm<T, std::void_t<decltype(T::kMaxCtasPerSm)>>
+    : std::integral_constant<uint32_t, (uint32_t)T::kMaxCtasPerSm> {};
+
 template <class T, class = void>
 struct has_dynamic_total : std::false_type {};
 template <class T>

@@ -53,6 +53,7 @@ struct Kernel {
   int num_regs;
   int static_smem;
   int occ_p, occ_n;
+  uint32_t max_per_sm;   // useful occupancy cap (0 = none)
   uint32_t threads() const { return block.x * block.y * block.z; }
 };
 
@@ -268,10 +269,15 @@ int refresh_done(accel_ctx* ctx, Request* r) {
 }
 
 
+// The solver's upper bound on a kernel's CTAs is its grid (PAPER.md lines
+// 538-541: work-groups are added "until resource saturation"), lowered to the
+// kernel's declared useful occupancy x SMs when it has one (R-solver-9).
 int demand_for(accel_ctx* ctx, const Step& s, uint32_t weight, accel_demand* d) {
   const Kernel& k = ctx->kernels[s.kid];
+  uint32_t cap = s.total;
+  if (k.max_per_sm) cap = std::min<uint64_t>(cap, (uint64_t)k.max_per_sm * (uint32_t)ctx->caps.sms);
   return accel_demand_of(&ctx->caps, k.threads(), (uint32_t)k.num_regs,
-                         (uint32_t)(k.static_smem + k.dyn_smem), s.total, weight, d);
+                         (uint32_t)(k.static_smem + k.dyn_smem), cap, weight, d);
 }
 
 int fetch_result(accel_ctx* ctx, Request* r) {
@@ -908,6 +914,8 @@ int accel_kernel_register(accel_ctx* ctx, const accel_kernel_desc* d, int32_t* k
   k.dyn_smem = d->dyn_smem;
   k.chunk = d->chunk ? d->chunk : 1;
   k.args_size = d->args_size;
+  // ACCEL_NO_OCC_CAP=1: ignore the useful-occupancy caps (A/B measurements)
+  k.max_per_sm = std::getenv("ACCEL_NO_OCC_CAP") ? 0u : d->max_ctas_per_sm;
   cudaFuncAttributes a;
   CK(ctx, cudaFuncGetAttributes(&a, k.pfn));
   if ((int)k.threads() > a.maxThreadsPerBlock) return ctx->fail(ACCEL_ENOFIT, "block larger than the kernel allows");

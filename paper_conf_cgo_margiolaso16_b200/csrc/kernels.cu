@@ -97,6 +97,7 @@ accel_kernel_desc make_desc(const char* name) {
   d.regs = 0;
   d.chunk = T::kChunk;
   d.args_size = sizeof(typename T::Args);
+  d.max_ctas_per_sm = max_ctas_per_sm<T>::value;
   if constexpr (has_vg_cost<T>::value)
     d.order_fn = reinterpret_cast<const void*>(&accel_lpt_order<T>);
   else

@@ -91,11 +91,22 @@ struct HistoT {
     }
     __syncthreads();
     uint32_t* gh = a.hist + (r & 1u) * bins;
+    // packed, even bin count: bins 2b and 2b+1 are one 8-B-aligned pair of
+    // global counters, flushed with ONE 64-bit atomic (half the L2 atomics:
+    // the flush is what an L2-bound co-runner competes with).  A count never
+    // reaches 2^32 (n < 2^32), so the low half cannot carry into the high one.
+    const bool pair64 = kPacked && (bins & 1u) == 0u;
     for (uint32_t b = threadIdx.x; b < words; b += kThreads) {
       const uint32_t c = h[b];
       if constexpr (kPacked) {
-        if (c & 0xffffu) atomicAdd(&gh[2 * b], c & 0xffffu);
-        if (c >> 16) atomicAdd(&gh[2 * b + 1], c >> 16);   // bin 2b+1 < bins whenever counted
+        if (pair64) {
+          if (c)
+            atomicAdd(reinterpret_cast<unsigned long long*>(gh + 2 * b),
+                      ((unsigned long long)(c >> 16) << 32) | (c & 0xffffu));
+        } else {
+          if (c & 0xffffu) atomicAdd(&gh[2 * b], c & 0xffffu);
+          if (c >> 16) atomicAdd(&gh[2 * b + 1], c >> 16);   // bin 2b+1 < bins whenever counted
+        }
       } else {
         if (c) atomicAdd(&gh[b], c);
       }

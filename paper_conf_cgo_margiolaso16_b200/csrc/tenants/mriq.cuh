@@ -36,6 +36,9 @@ struct MriqQ {
   static constexpr int kTile = 256;
   static constexpr uint32_t kChunk = 1;
   static constexpr int kMinBlocks = 6;
+  // useful occupancy (scripts/occ_scaling.py, isolated SHARED-static):
+  // 5.83 ms at 2 CTAs/SM = 5.80 ms at 3..6 -- issue-bound beyond 16 warps
+  static constexpr uint32_t kMaxCtasPerSm = 2;
   static constexpr uint32_t kDynSmem = 4 * kTile * sizeof(float);
 
   static __device__ __forceinline__ float frac_prod(float k, float x, float& err) {
@@ -45,10 +48,11 @@ struct MriqQ {
   }
 
   static __device__ __forceinline__ void body(const Args& a, const VirtualBlock& vb, char* smem) {
-    float* skx = reinterpret_cast<float*>(smem);
-    float* sky = skx + kTile;
-    float* skz = sky + kTile;
-    float* spm = skz + kTile;
+    // (kx, ky, kz, phiMag) of a k-sample packed in one 16-B slot: the inner
+    // loop issues ONE broadcast LDS.128 per sample instead of four LDS.32.
+    // Measured: with four, mri-q's 24 warps/SM kept the LSU queue full and a
+    // latency-bound co-runner on the same SM (bfs) ran 10x slower.
+    float4* sk = reinterpret_cast<float4*>(smem);
     const int t = threadIdx.x;
     const uint32_t v = vb.linear * kThreads + t;
     const bool have = v < a.numx;
@@ -60,24 +64,21 @@ struct MriqQ {
     for (uint32_t k0 = 0; k0 < a.numk; k0 += kTile) {
       __syncthreads();
       const uint32_t k = k0 + t;
-      if (k < a.numk) {
-        skx[t] = __ldg(a.kx + k);
-        sky[t] = __ldg(a.ky + k);
-        skz[t] = __ldg(a.kz + k);
-        spm[t] = __ldcg(a.phimag + k);   // written by the previous launch
-      }
+      if (k < a.numk)   // phiMag was written by the previous launch (L2)
+        sk[t] = make_float4(__ldg(a.kx + k), __ldg(a.ky + k), __ldg(a.kz + k), __ldcg(a.phimag + k));
       __syncthreads();
       const int n = min(kTile, (int)(a.numk - k0));
 #pragma unroll 4
       for (int j = 0; j < n; ++j) {
+        const float4 kj = sk[j];
         float err = 0.f;
-        const float f = frac_prod(skx[j], x, err) + frac_prod(sky[j], y, err) + frac_prod(skz[j], z, err);
+        const float f = frac_prod(kj.x, x, err) + frac_prod(kj.y, y, err) + frac_prod(kj.z, z, err);
         float tt = f + err;
         tt -= rintf(tt);                 // turns in [-0.5, 0.5]
         float s, c;
         __sincosf(two_pi * tt, &s, &c);
-        qr = fmaf(spm[j], c, qr);
-        qi = fmaf(spm[j], s, qi);
+        qr = fmaf(kj.w, c, qr);
+        qi = fmaf(kj.w, s, qi);
       }
     }
     if (have) {

@@ -226,6 +226,8 @@ class HistoJob(Job):
         self.n, self.bins, self.iters, self.sb = d["n"], d["bins"], d["iters"], d["sample_bytes"]
         if not (1 <= self.bins <= 16384 and (self.sb == 4 or self.bins == 256)):
             raise ValueError("histo: 1..16384 bins; u8 samples need 256 bins")
+        if self.n >= 1 << 32:
+            raise ValueError("histo: n < 2^32 samples (u32 counters)")
         # > 4096 bins: the packed 16-bit private histogram (VGs < 65536 samples)
         self.kernel = "histo" if self.bins <= 4096 else "histo_wide"
         # samples per VG: histo_wide flushes up to 16K bins per VG with global

@@ -25,6 +25,9 @@ jobs = [make_job(t, inputs[t]) for t in tenants]
 m, p = {"native": (abi.MODE_NATIVE, abi.POLICY_STATIC), "static": (abi.MODE_SHARED, abi.POLICY_STATIC),
         "resolve": (abi.MODE_SHARED, abi.POLICY_RESOLVE)}[mode]
 acc = Accel(0, mode=m, policy=p)
+for j in jobs:
+    if hasattr(j, "fit_levels"):
+        j.fit_levels(acc)
 for rep in range(3):
     ids = acc.submit(jobs)
     acc.sync()
@@ -36,7 +39,7 @@ for t, s, l in zip(tenants, st, ls):
     print(f"{t:8s} T(s)={s.elapsed_ms:7.3f} ms start={(s.first_start_ns - t0) / 1e3:8.1f} "
           f"end={(s.last_end_ns - t0) / 1e3:8.1f} us q0={s.quota_initial} qmin={s.quota_min} "
           f"qmax={s.quota_max} resolves={s.resolves}")
-    step = max(1, len(l) // 12)
+    step = max(1, len(l) // int(os.environ.get("TL_LINES", "12")))
     for i in range(0, len(l), step):
         x = l[i]
         print(f"    launch {i:3d}: {(x.t_first_ns - t0) / 1e3:8.1f} .. {(x.t_last_ns - t0) / 1e3:8.1f} us "

@@ -87,3 +87,12 @@ def test_pure_host_functions_validate():
     assert e.value.code == abi.ACCEL_ENOFIT
     with pytest.raises(abi.AccelError):
         abi.accel_metrics([1.0, 0.0], [1.0, 1.0])
+
+
+def test_useful_occupancy_caps():
+    """kMaxCtasPerSm reaches the descriptor (0 = no cap) -- values measured
+    with scripts/occ_scaling.py, R-solver-9."""
+    from paper_conf_cgo_margiolaso16_b200 import abi
+    want = {"mriq_q": 2, "histo_wide": 0, "histo": 0, "bfs": 3, "spmv": 4, "tpacf": 4, "stencil": 0, "cutcp": 0}
+    for n, v in want.items():
+        assert abi.accel_builtin_kernel(n).max_ctas_per_sm == v, n
