@@ -114,14 +114,17 @@ typedef struct {
   const void *order_fn;       /* host stub of accel_lpt_order<T>: the kernel's
                                  dequeue-order cost model (T::vg_cost); NULL =
                                  none (linear dequeue order)                    */
-  uint32_t max_ctas_per_sm;   /* useful occupancy (T::kMaxCtasPerSm): the kernel
-                                 gains nothing from more resident CTAs per SM
-                                 (measured, scripts/occ_scaling.py), so the
-                                 solver never gives it more than this x SMs --
-                                 the paper's greedy fill "until resource
-                                 saturation" stops at
-                                 the kernel's own saturation and the rest goes
-                                 to its co-runners.  0 = no cap.  SHARED only. */
+  uint32_t max_ctas_per_sm;   /* useful occupancy (T::kMaxCtasPerSm): the fewest
+                                 resident CTAs per SM at which the kernel alone
+                                 reaches >= 90 % of its full-device speed
+                                 (measured, scripts/occ_scaling.py).  While the
+                                 request shares the device the solver gives it
+                                 at most this x SMs -- the paper's greedy fill
+                                 "until resource saturation" (PAPER.md lines
+                                 538-541) stops at the kernel's own saturation
+                                 and the rest goes to its co-runners; alone it
+                                 keeps its full share.  0 = no cap.  SHARED
+                                 only (DESIGN.md R-solver-10). */
 } accel_kernel_desc;
 
 /* Fill *out with a built-in tenant kernel: "mop", "stencil", "histo", "bfs",
@@ -308,6 +311,16 @@ int accel_metrics(const double *ta, const double *ts, int32_t k, accel_mix_metri
  * ws_out[k] may be NULL. */
 int accel_metrics_weighted(const double *ta, const double *ts, const double *w, int32_t k, double *wunfairness,
                            double *ws_out);
+/* Profile-guided sharing ratios (DESIGN.md R-solver-11; PAPER.md lines
+ * 388-393 "changing the sharing ratio"): k requests, each with its isolated
+ * time ms[i*nf + j] when given the device fraction fracs[j] (fracs[0] = 1,
+ * strictly decreasing, > 0; scripts/share_profile.py measures them).  Writes
+ * the integer ratios w_out[k] (1..scale) that equalise the predicted slowdowns
+ * T_i(f_i)/T_i(1) under sum f_i = 1, and (if s_pred != NULL) the predicted
+ * slowdown of each request.  Pass w_out as accel_request.weight.  Pure host
+ * function.  ACCEL_EINVAL for invalid profiles. */
+int accel_guided_weights(int32_t k, int32_t nf, const double *fracs, const double *ms, uint32_t scale,
+                         uint32_t *w_out, double *s_pred);
 /* Encode a 2-D TMA tensor map (CUtensorMap, 128 B written to out128) for a
  * row-major fp32 matrix: `inner` elements per row (contiguous), `outer` rows,
  * rows row_stride_bytes apart (multiple of 16), box box_inner x box_outer,

@@ -44,7 +44,9 @@ typedef struct {
  * (r == 0 ? a0 : buf[(r-1)&1]) and writes buf[r&1]; after T launches the
  * result is in buf[(T-1)&1].  Interior: c1*(6-neighbour sum) - c0*a;
  * faces copy the input.  a0/buf0/buf1: DEVICE pointers to nx*ny*nz floats,
- * 16-B aligned, no padding required. */
+ * 16-B aligned, no padding required.
+ * Kernel "stencil2" (same arguments, nx % 4 == 0): VG tile 128 x 16 x 8, two
+ * rows per warp -- grid (ceil(nx/128), ceil(ny/16), ceil(nz/8)). */
 typedef struct {
   const float *a0;
   float *buf0;

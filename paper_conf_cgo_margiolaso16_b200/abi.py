@@ -161,6 +161,7 @@ class accel_sgemm_tc_args(C.Structure):
 accel_stencil_x_args = accel_stencil_args
 accel_sgemm_tc1_args = accel_sgemm_tc_args
 accel_stencil_deep_args = accel_stencil_args
+accel_stencil2_args = accel_stencil_args
 accel_stencil_bulk_args = accel_stencil_tma_args
 accel_histo_wide_args = accel_histo_args
 
@@ -208,7 +209,7 @@ EXPORTS = [
     "accel_init", "accel_finalize", "accel_set_mode", "accel_last_error", "accel_builtin_kernel",
     "accel_builtin_count", "accel_builtin_name", "accel_kernel_register", "accel_kernel_info_get",
     "accel_submit", "accel_submit_group", "accel_sync", "accel_epoch", "accel_stats", "accel_release",
-    "accel_tenant_stream", "accel_launch_times", "accel_launch_stats", "accel_vg_trace", "accel_demand_of", "accel_solve", "accel_placement_order", "accel_dequeue_order", "accel_metrics", "accel_metrics_weighted", "accel_overlap", "accel_tma_map_2d", "accel_tma_map_3d",
+    "accel_tenant_stream", "accel_launch_times", "accel_launch_stats", "accel_vg_trace", "accel_demand_of", "accel_solve", "accel_placement_order", "accel_dequeue_order", "accel_metrics", "accel_metrics_weighted", "accel_guided_weights", "accel_overlap", "accel_tma_map_2d", "accel_tma_map_3d",
 ]
 
 
@@ -249,6 +250,7 @@ def _load() -> C.CDLL:
         "accel_placement_order": (i32, [P(accel_caps), P(accel_demand), i32, P(i32)]),
         "accel_dequeue_order": (i32, [vp, i32, P(accel_dim3), vp, u32, vp]),
         "accel_metrics_weighted": (i32, [P(f64), P(f64), P(f64), i32, P(f64), P(f64)]),
+        "accel_guided_weights": (i32, [i32, i32, P(f64), P(f64), u32, P(u32), P(f64)]),
         "accel_metrics": (i32, [P(f64), P(f64), i32, P(accel_mix_metrics)]),
         "accel_overlap": (i32, [P(f64), P(f64), i32, P(f64)]),
         "accel_tma_map_2d": (i32, [vp, vp, u64, u64, u64, u32, u32, i32]),
@@ -431,6 +433,19 @@ def accel_metrics_weighted(ta: list[float], ts: list[float], w: list[float]) -> 
     ws = (f64 * max(k, 1))()
     check(lib.accel_metrics_weighted(arr(ta), arr(ts), arr(w), k, C.byref(wu), ws))
     return wu.value, list(ws)[:k]
+
+
+def accel_guided_weights(fracs: list[float], ms: list[list[float]], scale: int = 16) -> tuple[list[int], list[float]]:
+    """Profile-guided sharing ratios (DESIGN.md R-solver-11): ms[i][j] =
+    isolated time of request i at device fraction fracs[j].  Returns
+    (weights, predicted slowdowns)."""
+    k, nf = len(ms), len(fracs)
+    fr = (f64 * max(nf, 1))(*fracs)
+    flat = (f64 * max(k * nf, 1))(*[x for row in ms for x in row])
+    w = (u32 * max(k, 1))()
+    sp = (f64 * max(k, 1))()
+    check(lib.accel_guided_weights(k, nf, fr, flat, scale, w, sp))
+    return list(w)[:k], list(sp)[:k]
 
 
 def accel_overlap(start: list[float], end: list[float]) -> float:

@@ -270,12 +270,13 @@ int refresh_done(accel_ctx* ctx, Request* r) {
 
 
 // The solver's upper bound on a kernel's CTAs is its grid (PAPER.md lines
-// 538-541: work-groups are added "until resource saturation"), lowered to the
-// kernel's declared useful occupancy x SMs when it has one (R-solver-9).
-int demand_for(accel_ctx* ctx, const Step& s, uint32_t weight, accel_demand* d) {
+// 538-541: work-groups are added "until resource saturation"), lowered -- when
+// the request shares the device (in_mix) -- to the kernel's declared useful
+// occupancy x SMs (R-solver-10).  Alone, a request keeps its full share.
+int demand_for(accel_ctx* ctx, const Step& s, uint32_t weight, accel_demand* d, bool in_mix = false) {
   const Kernel& k = ctx->kernels[s.kid];
   uint32_t cap = s.total;
-  if (k.max_per_sm) cap = std::min<uint64_t>(cap, (uint64_t)k.max_per_sm * (uint32_t)ctx->caps.sms);
+  if (in_mix && k.max_per_sm) cap = std::min<uint64_t>(cap, (uint64_t)k.max_per_sm * (uint32_t)ctx->caps.sms);
   return accel_demand_of(&ctx->caps, k.threads(), (uint32_t)k.num_regs,
                          (uint32_t)(k.static_smem + k.dyn_smem), cap, weight, d);
 }
@@ -643,7 +644,7 @@ int assign_quotas(accel_ctx* ctx, std::vector<std::unique_ptr<Request>>& fresh) 
   std::vector<accel_demand> ds(order.size());
   for (size_t i = 0; i < order.size(); ++i) {
     Request* r = order[i];
-    int rc = demand_for(ctx, r->steps[r->main_step], r->weight, &ds[i]);
+    int rc = demand_for(ctx, r->steps[r->main_step], r->weight, &ds[i], order.size() > 1);
     if (rc) return ctx->fail(rc, "kernel does not fit on an SM");
   }
   std::vector<uint32_t> q(order.size());
@@ -666,7 +667,7 @@ int assign_quotas(accel_ctx* ctx, std::vector<std::unique_ptr<Request>>& fresh) 
         // R-solver-8: a secondary step is solved against the same active set,
         // with this request represented by the step's own kernel
         std::vector<accel_demand> dsj = ds;
-        rc = demand_for(ctx, s, r->weight, &dsj[i]);
+        rc = demand_for(ctx, s, r->weight, &dsj[i], order.size() > 1);
         if (rc) return ctx->fail(rc, "kernel does not fit on an SM");
         std::vector<uint32_t> qj(order.size());
         rc = accel_solve(&ctx->caps, dsj.data(), (int32_t)dsj.size(), qj.data());

@@ -115,6 +115,7 @@ const Builtin kBuiltins[] = {
     {"stencil", &make_desc<Stencil>},
     {"stencil_x", &make_desc<StencilX>},
     {"stencil_deep", &make_desc<StencilDeep>},
+    {"stencil2", &make_desc<Stencil2>},
     {"stencil_tma", &make_desc<StencilTma>},
     {"stencil_bulk", &make_desc<StencilBulk>},
     {"histo", &make_desc<Histo>},

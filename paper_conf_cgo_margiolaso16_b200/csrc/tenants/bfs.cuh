@@ -20,9 +20,10 @@ struct Bfs {
   static constexpr int kThreads = 256;
   static constexpr uint32_t kChunk = 1;
   static constexpr int kMinBlocks = 6;
-  // useful occupancy: 0.373 ms at 3 CTAs/SM vs 0.42 ms at 6 (more CTAs only
-  // add queue-append contention on the small levels; scripts/occ_scaling.py)
-  static constexpr uint32_t kMaxCtasPerSm = 3;
+  // useful occupancy in a mix (R-solver-10): 0.374 ms at 2 CTAs/SM, 0.373 at
+  // 3, 0.42 at 6 (more CTAs only add queue-append contention on the small
+  // levels; scripts/occ_scaling.py)
+  static constexpr uint32_t kMaxCtasPerSm = 2;
   static constexpr uint32_t kQueueCap = 4096;  // local queue entries (16 KB)
   static constexpr uint32_t kDynSmem = kQueueCap * sizeof(int32_t);
   static constexpr bool kDynamicTotal = true;

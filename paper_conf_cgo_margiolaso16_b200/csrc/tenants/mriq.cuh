@@ -36,9 +36,11 @@ struct MriqQ {
   static constexpr int kTile = 256;
   static constexpr uint32_t kChunk = 1;
   static constexpr int kMinBlocks = 6;
-  // useful occupancy (scripts/occ_scaling.py, isolated SHARED-static):
-  // 5.83 ms at 2 CTAs/SM = 5.80 ms at 3..6 -- issue-bound beyond 16 warps
-  static constexpr uint32_t kMaxCtasPerSm = 2;
+  // useful occupancy in a mix (R-solver-10; scripts/occ_scaling.py, isolated
+  // SHARED-static): 6.34 ms at 1 CTA/SM = 92 % of the 5.80 ms at 3..6 -- one
+  // CTA per SM nearly saturates the issue slots; its 2nd..6th CTA would take
+  // them from a co-runner on the same SM (bfs next to 3 mri-q CTAs/SM: 12x)
+  static constexpr uint32_t kMaxCtasPerSm = 1;
   static constexpr uint32_t kDynSmem = 4 * kTile * sizeof(float);
 
   static __device__ __forceinline__ float frac_prod(float k, float x, float& err) {

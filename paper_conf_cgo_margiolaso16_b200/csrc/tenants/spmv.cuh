@@ -19,7 +19,7 @@ struct Spmv {
   static constexpr int kLanesPerRow = kThreads / kRows;  // 4
   static constexpr uint32_t kChunk = 1;
   static constexpr int kMinBlocks = 6;
-  static constexpr uint32_t kMaxCtasPerSm = 4;   // 1.21 ms at 4 CTAs/SM vs 1.26 at 6 (occ_scaling.py)
+  static constexpr uint32_t kMaxCtasPerSm = 4;   // in a mix: 1.21 ms at 4 CTAs/SM vs 1.26 at 6 (occ_scaling.py)
   static constexpr uint32_t kDynSmem = 0;
 
   static __device__ __forceinline__ void body(const Args& a, const VirtualBlock& vb, char*) {

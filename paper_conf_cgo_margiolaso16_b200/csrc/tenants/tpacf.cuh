@@ -33,7 +33,7 @@ struct Tpacf {
   static constexpr uint32_t kChunk = 1;
   static constexpr bool kSpread = true;     // VG cost varies in space (dispatch.cuh)
   static constexpr int kMinBlocks = 6;   // <= 40 regs: smem allows 6 CTAs/SM
-  static constexpr uint32_t kMaxCtasPerSm = 4;   // 1.385 ms at 4 CTAs/SM vs 1.40 at 6 (occ_scaling.py)
+  static constexpr uint32_t kMaxCtasPerSm = 3;   // in a mix: 1.414 ms at 3 CTAs/SM vs 1.40 at 6 (occ_scaling.py)
   static constexpr int kWarps = kThreads / 32;
   static constexpr int kMaxBins = 32;      // nedges + 1 <= 32
   static constexpr int kTile = 256;

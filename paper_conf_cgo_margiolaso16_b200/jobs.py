@@ -187,7 +187,6 @@ class StencilJob(Job):
         self.out = {"a": self.buf[(self.sweeps - 1) & 1]}
         self.args = abi.accel_stencil_args(self.inputs["a0"].data_ptr(), self.buf[0].data_ptr(),
                                            self.buf[1].data_ptr(), self.nx, self.ny, self.nz, d["c0"], d["c1"])
-        grid = (_cdiv(self.nx, self.TX), _cdiv(self.ny, self.TY), _cdiv(self.nz, self.TZ))
         # default: cp.async staging; stencil_tma is opt-in until its drift next to
         # bfs is understood (DESIGN.md §6 "stencil staging", scripts/diag_tma.py)
         kernel = kernel or d.get("kernel") or os.environ.get("ACCEL_STENCIL_KERNEL") or \
@@ -207,6 +206,8 @@ class StencilJob(Job):
                 self.gmaps = torch.frombuffer(bytearray(maps), dtype=torch.uint8).to(self.device)
                 self.args.gmaps = self.gmaps.data_ptr()
         self.kernel = kernel
+        ty = 16 if kernel == "stencil2" else self.TY   # stencil2: two rows per warp
+        grid = (_cdiv(self.nx, self.TX), _cdiv(self.ny, ty), _cdiv(self.nz, self.TZ))
         self.steps = [Step(kernel, grid, self.args, self.sweeps)]
 
     def result(self):

@@ -43,8 +43,20 @@ from paper_conf_cgo_margiolaso16_b200.runtime import Accel  # noqa: E402
 TENANTS = ["bfs", "cutcp", "stencil", "tpacf", "histo", "spmv", "sgemm", "mriq"]
 ALPHA = 0.0   # --alpha: SHARED-mode weights ~ T(a)^alpha (0 = equal shares, the paper's policy)
 MODES = [("native", abi.MODE_NATIVE, abi.POLICY_STATIC), ("resolve", abi.MODE_SHARED, abi.POLICY_RESOLVE),
-         ("static", abi.MODE_SHARED, abi.POLICY_STATIC)]
-SHARED = ["resolve", "static"]
+         ("static", abi.MODE_SHARED, abi.POLICY_STATIC), ("guided", abi.MODE_SHARED, abi.POLICY_RESOLVE)]
+SHARED = ["resolve", "static", "guided"]
+# "guided": RESOLVE with profile-guided sharing ratios (DESIGN.md R-solver-11)
+# from the measured share profiles (scripts/share_profile.py)
+PROFILE = os.path.join(ROOT, "profiles", "r2", "share_profile.json")
+_prof = None
+
+
+def guided_weights(names):
+    global _prof
+    if _prof is None:
+        _prof = json.load(open(PROFILE))
+    ms = [_prof["profile"][t]["ms"] for t in names]
+    return abi.accel_guided_weights(_prof["fracs"], ms)[0]
 
 
 def gm(xs):
@@ -85,7 +97,7 @@ class Runner:
             for i, (j, dl) in enumerate(zip(jobs, delays_s)):
                 while time.perf_counter() - t0 < dl:
                     pass
-                ids += self.acc.submit([j], tenants=[i])
+                ids += self.acc.submit([j], tenants=[i], weights=None if weights is None else [weights[i]])
         self.acc.sync()
         st = [self.acc.stats(i) for i in ids]
         self.acc.release()
@@ -126,7 +138,8 @@ def config3(r: Runner, ta, reps, only=None):
         jb = r.jobs[b][1] if a == b else r.jobs[b][0]
         res = {"mix": [a, b]}
         for name, mode, pol in MODES:
-            runs = [mix_metrics(r.run([ja, jb], mode, pol), [ta[a], ta[b]]) for _ in range(reps)]
+            w = guided_weights([a, b]) if name == "guided" else None
+            runs = [mix_metrics(r.run([ja, jb], mode, pol, weights=w), [ta[a], ta[b]]) for _ in range(reps)]
             res[name] = {k: statistics.mean(x[k] for x in runs) for k in ("U", "STP", "ANTT", "makespan_ms", "WANTT")}
         mixes.append(res)
         print(json.dumps({"mix": res["mix"], **{n: {k: round(v, 3) for k, v in res[n].items()} for n, _, _ in MODES}}),
@@ -155,7 +168,8 @@ def config4(r: Runner, ta, reps):
     tal = [ta[t] for t in order]
     out = {"order": order, "delta_ms": delta * 1e3}
     for name, mode, pol in MODES:
-        runs = [mix_metrics(r.run(jobs, mode, pol, delays), tal) for _ in range(reps)]
+        w = guided_weights(order) if name == "guided" else None
+        runs = [mix_metrics(r.run(jobs, mode, pol, delays, weights=w), tal) for _ in range(reps)]
         out[name] = {k: statistics.mean(x[k] for x in runs) for k in ("U", "STP", "ANTT", "WANTT", "makespan_ms")}
         out[name]["slowdowns"] = dict(zip(order, [statistics.mean(x["ts_ms"][i] for x in runs) / tal[i]
                                                   for i in range(len(order))]))
@@ -189,8 +203,8 @@ def sampled(r: Runner, ta, reps, k, n, seed, repeat=False):
             seen[t] = seen.get(t, 0) + 1
         res = {"mix": names}
         for name, mode, pol in MODES:
-            w = None
-            if ALPHA and mode == abi.MODE_SHARED:
+            w = guided_weights(names) if name == "guided" else None
+            if ALPHA and mode == abi.MODE_SHARED and name != "guided":
                 # profile-guided sharing ratio: w ~ T(a)^alpha (alpha < 0: the
                 # shorter requests get the larger shares)
                 tmax = max(ta[t] for t in names)

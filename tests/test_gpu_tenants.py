@@ -86,21 +86,22 @@ def test_mop_small_fullcaps(acc, oracle_lib):
                                        ("tiny", dict(nx=129, ny=8, nz=9, sweeps=2)),    # one column past a tile
                                        ("tiny", dict(nx=2, ny=5, nz=4, sweeps=2)),      # all faces
                                        ("small", dict(sweeps=10))])
-@pytest.mark.parametrize("kernel", ["default", "stencil_tma"])
+@pytest.mark.parametrize("kernel", ["default", "stencil_tma", "stencil", "stencil2"])
 def test_stencil(acc_tiny_caps, oracle_lib, size, over, kernel):
-    """default = the cp.async staging ("stencil") when nx % 4 == 0, stencil_x
-    otherwise; "stencil_tma" = the TMA ring (nx % 4 == 0 only)."""
+    """default = the job's choice for this nx; "stencil" (8 rows per tile),
+    "stencil2" (16 rows, two per warp) and "stencil_tma" (TMA ring) need
+    nx % 4 == 0."""
     from paper_conf_cgo_margiolaso16_b200.jobs import StencilJob
     d = synth.preset("stencil", size, **over)
-    if kernel == "stencil_tma" and d["nx"] % 4:
-        pytest.skip("TMA staging needs nx % 4 == 0")
+    if kernel != "default" and d["nx"] % 4:
+        pytest.skip(f"{kernel} needs nx % 4 == 0")
     k = None if kernel == "default" else kernel
     nat, sh, _ = run_modes(acc_tiny_caps, lambda: StencilJob(d, kernel=k))
     same(nat, sh)
     assert_close_fp32(sh["a"], oracle_lib.stencil(d), what="stencil")
 
 
-@pytest.mark.parametrize("kernel", ["stencil_tma", "stencil"])
+@pytest.mark.parametrize("kernel", ["stencil_tma", "stencil", "stencil2"])
 def test_stencil_default_sampled(acc, oracle_lib, kernel):
     """BASELINE size (512x512x64, 100 sweeps) in the bench's launch
     configuration; the oracle at full size is ~1.7e9 point-sweeps of plain C,
@@ -327,6 +328,9 @@ def _stencil_fp32_replica(d):
                                          ("stencil_bulk", dict(nx=136, ny=17, nz=19, sweeps=4)),
                                          ("stencil_bulk", dict(nx=260, ny=9, nz=8, sweeps=3)),
                                          ("stencil", dict(nx=136, ny=17, nz=19, sweeps=4)),
+                                         ("stencil2", dict(nx=136, ny=17, nz=19, sweeps=4)),
+                                         ("stencil2", dict(nx=260, ny=33, nz=8, sweeps=3)),
+                                         ("stencil2", dict(nx=4, ny=3, nz=3, sweeps=2)),
                                          ("stencil_x", dict(nx=70, ny=21, nz=19, sweeps=3))])
 def test_stencil_bit_exact_fp32_sequence(acc_tiny_caps, kernel, over):
     """Every stencil kernel computes the pinned fp32 round-to-nearest sequence
