@@ -396,16 +396,27 @@ def run_rank(args, rank, world, local, ranks: Ranks) -> dict:
 
     POL = {"resolve": abi.POLICY_RESOLVE, "static": abi.POLICY_STATIC}
     head_pol = POL[args.policy]
-    # reported beside the headline: STATIC (the paper's policy) and RESOLVE
+    # reported beside the headline: STATIC (the paper's policy) and RESOLVE,
+    # and "guided" -- RESOLVE with profile-guided sharing ratios (DESIGN.md
+    # R-solver-11) from the committed share profiles, when every tenant has one
     other_pols = [p for p in POL if p != args.policy]
+    WEIGHTS = {p: None for p in POL}
+    prof_path = os.path.join(ROOT, "profiles", "r2", "share_profile.json")
+    if os.path.exists(prof_path):
+        prof = json.load(open(prof_path))
+        if all(t in prof["profile"] for t in tenants):
+            POL["guided"] = abi.POLICY_RESOLVE
+            WEIGHTS["guided"] = abi.accel_guided_weights(prof["fracs"],
+                                                         [prof["profile"][t]["ms"] for t in tenants])[0]
+            other_pols.append("guided")
 
-    def run_group(js, mode, e2e=False, launch_events=False, policy=None):
+    def run_group(js, mode, e2e=False, launch_events=False, policy=None, weights=None):
         policy = head_pol if policy is None else policy
         if acc.mode != mode or acc.policy != policy:
             acc.set_mode(mode, policy)
         flush()
         acc.epoch()
-        ids = acc.submit(js, e2e=e2e, launch_events=launch_events)
+        ids = acc.submit(js, e2e=e2e, launch_events=launch_events, weights=weights)
         acc.sync()
         st = [acc.stats(i) for i in ids]
         lt = [acc.launch_times(i, j.launches()) for i, j in zip(ids, js)] if launch_events else None
@@ -423,7 +434,7 @@ def run_rank(args, rank, world, local, ranks: Ranks) -> dict:
         for name, mode, pol in [("native", abi.MODE_NATIVE, abi.POLICY_STATIC)] + \
                 [(p, abi.MODE_SHARED, POL[p]) for p in (args.policy, *other_pols)]:
             vacc.set_mode(mode, pol)
-            st = vacc.run(jobs)
+            st = vacc.run(jobs, weights=WEIGHTS.get(name))
             assert all(s.coverage_ok == 1 for s in st), f"coverage check failed ({name})"
             res = [j.result() for j in jobs]
             if ref is None:
@@ -453,8 +464,9 @@ def run_rank(args, rank, world, local, ranks: Ranks) -> dict:
                 iso_launch[j.name] = lts
     ta = [iso_native[t] for t in tenants]
 
-    def steps_loop(mode, k, e2e=False, policy=None):
-        return [run_group(jobs, mode, e2e=e2e, launch_events=True, policy=policy) for _ in range(k)]
+    def steps_loop(mode, k, e2e=False, policy=None, weights=None):
+        return [run_group(jobs, mode, e2e=e2e, launch_events=True, policy=policy, weights=weights)
+                for _ in range(k)]
 
     steps_loop(abi.MODE_SHARED, args.warmup)
     ranks.barrier()
@@ -467,8 +479,8 @@ def run_rank(args, rank, world, local, ranks: Ranks) -> dict:
     native = steps_loop(abi.MODE_NATIVE, args.steps)
     other = {}
     for p in other_pols:
-        steps_loop(abi.MODE_SHARED, 1, policy=POL[p])
-        other[p] = steps_loop(abi.MODE_SHARED, args.steps, policy=POL[p])
+        steps_loop(abi.MODE_SHARED, 1, policy=POL[p], weights=WEIGHTS[p])
+        other[p] = steps_loop(abi.MODE_SHARED, args.steps, policy=POL[p], weights=WEIGHTS[p])
     steps_loop(abi.MODE_SHARED, 1, e2e=True)
     e2e = steps_loop(abi.MODE_SHARED, args.steps, e2e=True)
 
@@ -531,6 +543,7 @@ def run_rank(args, rank, world, local, ranks: Ranks) -> dict:
     launches_per_step = sum(1 + join + j.launches() for j in jobs)
     res = {"rank": rank, "dev_ms": sum(sh["makespan_ms"]), "e2e_ms": sum(ee["makespan_ms"]),
            "nat_ms": sum(na["makespan_ms"]), "oth_ms": {p: sum(v["makespan_ms"]) for p, v in ot.items()},
+           "weights": {p: w for p, w in WEIGHTS.items() if w is not None},
            "tenants": tenants, "size": size, "sh": sh, "na": na, "ot": ot,
            "quotas": [[s.quota_initial, s.quota_min, s.quota_max, s.resolves] for s in shared[-1][0]],
            "clk": clk.summary(), "ta": ta, "iso_persist": [iso_persist[t] for t in tenants],
@@ -602,6 +615,8 @@ def result_line(args, allres, world, cpu) -> dict:
     antt_sh, antt_na, other_sum = agg["antt_sh"], agg["antt_na"], agg["other"]
     for p in other_sum:
         other_sum[p]["T_s_ms"] = dict(zip(tenants, np.mean(r0["ot"][p]["ts_ms"], 0).tolist()))
+        if p in r0.get("weights", {}):
+            other_sum[p]["weights"] = dict(zip(tenants, r0["weights"][p]))
     clocks = r0["clk"]
     dom = r0["dom"]
     roof = r0["roof"]
