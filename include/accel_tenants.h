@@ -155,7 +155,10 @@ typedef struct {
   unsigned long long *dd, *rr, *dr;
 } accel_tpacf_args;
 
-/* spmv -- y = A x, CSR fp32.  block 256, VG = 64 rows, grid ceil(n/64). */
+/* spmv -- y = A x, CSR fp32.  block 256, VG = 64 rows, grid ceil(n/64).
+ * Kernel "spmv_v4" (same arguments): 128-bit col/val loads in aligned
+ * 4-element chunks; col and val must be 16-B aligned and readable up to
+ * ceil(nnz/4)*4 elements (pad with anything: out-of-row elements are masked). */
 typedef struct {
   const int32_t *row_ptr;
   const int32_t *col;

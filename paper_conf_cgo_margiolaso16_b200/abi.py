@@ -160,6 +160,7 @@ class accel_sgemm_tc_args(C.Structure):
 # kernel variants that take the same argument struct
 accel_stencil_x_args = accel_stencil_args
 accel_sgemm_tc1_args = accel_sgemm_tc_args
+accel_spmv_v4_args = accel_spmv_args
 accel_stencil_deep_args = accel_stencil_args
 accel_stencil2_args = accel_stencil_args
 accel_stencil_bulk_args = accel_stencil_tma_args

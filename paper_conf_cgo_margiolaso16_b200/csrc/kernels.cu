@@ -126,6 +126,7 @@ const Builtin kBuiltins[] = {
     {"cutcp", &make_desc<Cutcp>},
     {"tpacf", &make_desc<Tpacf>},
     {"spmv", &make_desc<Spmv>},
+    {"spmv_v4", &make_desc<SpmvV4>},
     {"sgemm", &make_desc<Sgemm>},
     {"sgemm_split", &make_desc<SgemmSplit>},
     {"sgemm_tc", &make_desc<SgemmTc>},

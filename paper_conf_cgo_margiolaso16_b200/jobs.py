@@ -371,16 +371,25 @@ class TpacfJob(Job):
 
 
 class SpmvJob(Job):
-    def __init__(self, d: dict, device="cuda"):
+    """kernel "spmv_v4" (default; ACCEL_SPMV_KERNEL=spmv for the scalar one):
+    col/val padded to a multiple of 4 elements for the 128-bit chunk loads."""
+
+    def __init__(self, d: dict, device="cuda", kernel: str | None = None):
         super().__init__(name="spmv", device=torch.device(device))
         self.n, self.nnz, self.iters = d["n"], d["nnz"], d["iters"]
-        self.inputs = {k: _dev(d[k], self.device) for k in ("row_ptr", "col", "val", "x")}
+        self.kernel = kernel or os.environ.get("ACCEL_SPMV_KERNEL", "spmv_v4")
+        pad = (-self.nnz) % 4 if self.kernel == "spmv_v4" else 0
+        arrs = {k: d[k] for k in ("row_ptr", "col", "val", "x")}
+        if pad:
+            arrs["col"] = np.concatenate([arrs["col"], np.zeros(pad, arrs["col"].dtype)])
+            arrs["val"] = np.concatenate([arrs["val"], np.zeros(pad, arrs["val"].dtype)])
+        self.inputs = {k: _dev(v, self.device) for k, v in arrs.items()}
         self.y = torch.empty(self.n, dtype=torch.float32, device=self.device)
         self.out = {"y": self.y}
         i = self.inputs
         self.args = abi.accel_spmv_args(i["row_ptr"].data_ptr(), i["col"].data_ptr(), i["val"].data_ptr(),
                                         i["x"].data_ptr(), self.y.data_ptr(), self.n)
-        self.steps = [Step("spmv", (_cdiv(self.n, 64), 1, 1), self.args, self.iters)]
+        self.steps = [Step(self.kernel, (_cdiv(self.n, 64), 1, 1), self.args, self.iters)]
 
     def result(self):
         return {"y": _np(self.y, np.float32)}

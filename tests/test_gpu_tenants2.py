@@ -9,19 +9,23 @@ from tests.test_gpu_tenants import acc, acc_tiny_caps, run_modes, same  # noqa: 
 pytestmark = pytest.mark.gpu
 
 
-@pytest.mark.parametrize("size,over", [("tiny", {}), ("small", dict(iters=3)), ("tiny", dict(grid=7, reach=3))])
-def test_spmv(acc_tiny_caps, oracle_lib, size, over):
+@pytest.mark.parametrize("size,over", [("tiny", {}), ("small", dict(iters=3)), ("tiny", dict(grid=7, reach=3)),
+                                       ("tiny", dict(grid=5, reach=1))])
+@pytest.mark.parametrize("kernel", ["spmv", "spmv_v4"])
+def test_spmv(acc_tiny_caps, oracle_lib, size, over, kernel):
+    """spmv_v4: 128-bit chunk loads over padded col/val (any nnz % 4)."""
     from paper_conf_cgo_margiolaso16_b200.jobs import SpmvJob
     d = synth.preset("spmv", size, **over)
-    nat, sh, _ = run_modes(acc_tiny_caps, lambda: SpmvJob(d))
+    nat, sh, _ = run_modes(acc_tiny_caps, lambda: SpmvJob(d, kernel=kernel))
     same(nat, sh)
     assert_close_fp32(sh["y"], oracle_lib.spmv(d), what="spmv")
 
 
-def test_spmv_default(acc, oracle_lib):
+@pytest.mark.parametrize("kernel", ["spmv", "spmv_v4"])
+def test_spmv_default(acc, oracle_lib, kernel):
     from paper_conf_cgo_margiolaso16_b200.jobs import SpmvJob
     d = synth.preset("spmv", "default", iters=2)
-    nat, sh, _ = run_modes(acc, lambda: SpmvJob(d))
+    nat, sh, _ = run_modes(acc, lambda: SpmvJob(d, kernel=kernel))
     same(nat, sh)
     assert_close_fp32(sh["y"], oracle_lib.spmv(d), what="spmv default")
 
