@@ -371,13 +371,16 @@ class TpacfJob(Job):
 
 
 class SpmvJob(Job):
-    """kernel "spmv_v4" (default; ACCEL_SPMV_KERNEL=spmv for the scalar one):
-    col/val padded to a multiple of 4 elements for the 128-bit chunk loads."""
+    """kernel "spmv" (default) or "spmv_v4" (ACCEL_SPMV_KERNEL=spmv_v4: 128-bit
+    chunk loads over col/val padded to a multiple of 4 elements).  spmv_v4 is
+    22 % faster natively but only 7 % in SHARED mode (2-us VGs: the per-VG
+    hand-over of the persistent loop shows), which made the sampled mixes less
+    fair (its T(a) fell more than its shared time) -- DESIGN.md §6."""
 
     def __init__(self, d: dict, device="cuda", kernel: str | None = None):
         super().__init__(name="spmv", device=torch.device(device))
         self.n, self.nnz, self.iters = d["n"], d["nnz"], d["iters"]
-        self.kernel = kernel or os.environ.get("ACCEL_SPMV_KERNEL", "spmv_v4")
+        self.kernel = kernel or os.environ.get("ACCEL_SPMV_KERNEL", "spmv")
         pad = (-self.nnz) % 4 if self.kernel == "spmv_v4" else 0
         arrs = {k: d[k] for k in ("row_ptr", "col", "val", "x")}
         if pad:
