@@ -10,7 +10,8 @@ import ctypes as C
 import os
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(_HERE, "libaccel.so")
+# ACCEL_LIB: load another build of the same ABI (A/B measurements only)
+LIB_PATH = os.environ.get("ACCEL_LIB") or os.path.join(_HERE, "libaccel.so")
 
 ACCEL_OK = 0
 ACCEL_EINVAL = -1

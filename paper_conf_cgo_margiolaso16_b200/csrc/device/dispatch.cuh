@@ -33,10 +33,25 @@
 // admission and the first dequeue are ONE atomic (and every dequeue returns a
 // fresh alive count for free).  Growing adds CTAs -- sticky top-up grids launched by the
 // host monitor on the tenant's second stream, which serve the current launch
-// and then follow the request's later launches.  Because a top-up CTA may
-// still run VGs of launch l after launch l's main grid retired, a launch whose
-// predecessor was topped up first waits for it to complete (queue exhausted
-// and no CTA alive) -- a wait on already-running CTAs only, so no deadlock.
+// and then follow the request's later launches.
+//
+// Completion accounting (who waits for whom).  Launch l+1's main grid and the
+// request's join kernel follow launch l's main grid in stream order
+// (griddepcontrol.wait / the kernel boundary), so they only need launch l's
+// TOP-UP CTAs to be done: a top-up CTA counts itself in `tu_alive` before it
+// joins a launch and leaves it with a release fence + decrement
+// (wait_topups).  A top-up CTA is in no stream order with the main grids:
+// before it serves launch l+1 it needs launch l complete (wait_hybrid).  Main
+// CTAs that saw the launch `topped` at their last dequeue retire with a
+// release fence and the `alive` decrement, so a topped launch completes as
+// soon as its last CTA leaves (alive == 0); a main CTA of a launch no top-up
+// had joined retires with no fence and no atomic -- the single-tenant case --
+// and a top-up that joins such a launch late falls back to waiting until
+// launch l+1's main grid has STARTED (ctl->cur, a release by the CTA holding
+// l+1's first ticket after its griddepcontrol.wait: l's main grid is then
+// complete) and l's top-ups are done.  An early main grid (R-place-3,
+// launched ahead on a side stream) waits for its predecessor's main CTAs too:
+// that request's launches carry kCfgAccount (every main CTA accounts).
 #pragma once
 
 #include <cstdint>
@@ -98,7 +113,7 @@ struct alignas(128) Desc {
   unsigned long long t_last;   // max %globaltimer over CTA ends
   uint32_t total_seen;   // total as read by the CTAs (dynamic for bfs)
   uint32_t ctas_started; // CTAs admitted with work
-  uint32_t pad_alive;
+  uint32_t tu_alive;     // RESOLVE: top-up CTAs in this launch (wait_topups)
   uint32_t max_alive;    // high-water mark of `alive` (RESOLVE)
   uint32_t topped;       // a top-up CTA joined this launch (RESOLVE)
   uint32_t admit_fail;   // RESOLVE: CTAs admitted over the live quota (ran one chunk, left)
@@ -255,6 +270,7 @@ constexpr uint32_t kTerminate = 0xffffffffu;
 
 // A launch is complete when its queue is exhausted and no CTA is admitted
 // (a CTA is admitted before its first dequeue and leaves after its last VG).
+// Used only where every CTA of the launch accounts (kCfgAccount requests).
 __device__ __forceinline__ void wait_complete(const Desc* p) {
   for (;;) {
     const uint32_t tot = ld_volatile(&p->total_seen);
@@ -268,6 +284,49 @@ __device__ __forceinline__ void wait_complete(const Desc* p) {
   fence_acq_rel();
   // the launch's results were written through the generic proxy by other CTAs;
   // this CTA may read them with TMA (async proxy)
+  asm volatile("fence.proxy.async.global;" ::: "memory");
+}
+
+// Top-up CTA: wait until launch p (the predecessor of request launch
+// `next_idx`) is complete -- every admitted CTA left (alive == 0: all of p's
+// main CTAs accounted because p was topped), or p's successor main grid has
+// started (p's main grid done) and p's own top-ups are done.
+__device__ __forceinline__ void wait_hybrid(const Desc* p, uint32_t next_idx) {
+  for (;;) {
+    const uint32_t tot = ld_volatile(&p->total_seen);
+    const unsigned long long v = ld_volatile_u64(&p->qa);
+    if (tot != kTerminate && qa_next(v) >= tot) {
+      if (qa_alive(v) == 0) {
+        fence_acq_rel();
+        if (ld_volatile(&p->draining) == 0) break;
+      }
+      if (ld_volatile(&p->ctl->cur) >= next_idx) {
+        fence_acq_rel();
+        if (ld_volatile(&p->tu_alive) == 0 && ld_volatile(&p->draining) == 0) break;
+      }
+    }
+    __nanosleep(256);
+  }
+  fence_acq_rel();
+  asm volatile("fence.proxy.async.global;" ::: "memory");
+}
+
+// Launch p's main grid is known complete (stream order, or ctl->cur past it):
+// wait until its top-up CTAs are done too.  The queue word is read first: a
+// top-up that joined before the queue ran dry counted itself in tu_alive
+// before its admission atomic (release fence in between), so it is visible
+// here; one that joins later gets no VG.
+__device__ __forceinline__ void wait_topups(const Desc* p) {
+  for (;;) {
+    const uint32_t tot = ld_volatile(&p->total_seen);
+    const unsigned long long v = ld_volatile_u64(&p->qa);
+    if (tot != kTerminate && qa_next(v) >= tot) {
+      fence_acq_rel();
+      if (ld_volatile(&p->tu_alive) == 0 && ld_volatile(&p->draining) == 0) break;
+    }
+    __nanosleep(256);
+  }
+  fence_acq_rel();
   asm volatile("fence.proxy.async.global;" ::: "memory");
 }
 
@@ -287,6 +346,9 @@ enum : uint32_t {
   kCfgStaticFirst = 1u << 19,  // main grid: CTA b's first chunk is [b*chunk, (b+1)*chunk)
                                // with no atomic (desc_init starts the queue head at
                            // grid*chunk and, under RESOLVE, `alive` at grid)
+  kCfgAccount = 1u << 21,  // RESOLVE main grid whose CTAs retire with the fenced `alive`
+                           // decrement (a request with an early main grid, R-place-3)
+  kCfgTopup = 1u << 22,    // a top-up CTA (accel_topup): always accounts
   // measurement-only ablations (env ACCEL_ABLATE on the host; scripts/isolated.py)
   kAblNoFence = 1u << 24,  // retire without the release fence (UNSAFE with top-ups)
   kAblNoLive = 1u << 25,   // never load the live quota (no shrink)
@@ -324,6 +386,7 @@ struct SchedState {
   // latency in front of the queue atomic
   uint32_t hint_live, hint_alive;
   uint8_t have_nxt, admitted, draining;
+  uint8_t top_seen;    // RESOLVE: the launch was topped at this CTA's last dequeue
   uint8_t over;        // RESOLVE: admitted over the live quota -> leave at the next dequeue
   uint8_t long_vg;     // the last VG ran longer than kLongVgNs
   template <bool kSpread>
@@ -393,13 +456,21 @@ __device__ __forceinline__ unsigned long long dequeue(Desc* d, SchedState* S) {
 
 template <bool kResolve>
 __device__ __forceinline__ void retire(Desc* d, uint32_t cfg, const SchedState* S) {
-  if (kResolve && S->admitted) {
-    if (!(cfg & kAblNoFence)) fence_acq_rel();  // this CTA's VG results before the alive decrement
-    if (!(cfg & kAblNoDec)) atomicAdd(&d->qa, kAliveNeg);
-  }
-  if (kResolve && S->draining) {
-    fence_acq_rel();  // the last VG's results before the draining decrement
-    atomicSub(&d->draining, 1u);
+  if (kResolve) {
+    // a main-grid CTA that ran until the queue was dry retires silently: its
+    // results reach its waiters through stream order (see the header)
+    if (S->admitted && ((cfg & (kCfgAccount | kCfgTopup)) || S->top_seen)) {
+      if (!(cfg & kAblNoFence)) fence_acq_rel();  // this CTA's VG results before the alive decrement
+      if (!(cfg & kAblNoDec)) atomicAdd(&d->qa, kAliveNeg);
+    }
+    if (S->draining) {
+      fence_acq_rel();  // the last VG's results before the draining decrement
+      atomicSub(&d->draining, 1u);
+    }
+    if (cfg & kCfgTopup) {
+      fence_acq_rel();
+      atomicSub(&d->tu_alive, 1u);
+    }
   }
   if (cfg & kCfgStamps) red_max_u64(&d->t_last, globaltimer());
 }
@@ -416,6 +487,7 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     S->admitted = 1;
     S->draining = 0;
     S->over = 0;
+    S->top_seen = 1;   // (conservative until the first dynamic dequeue)
     // Static first chunk (main grids): measured, the first dequeue of 740
     // CTAs on one queue word serialised in L2 and spread the CTAs' first VG
     // starts over 6 us of a 30-us stencil launch (scripts/vg_trace.py)
@@ -458,26 +530,32 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
           d->last_live = live;
         }
       }
-      // the CTA holding the launch's first ticket announces it to top-up grids
-      if (b == 0) asm volatile("red.relaxed.gpu.global.max.u32 [%0], %1;" ::"l"(&d->ctl->cur), "r"(d->req_idx) : "memory");
+      // the CTA holding the launch's first ticket announces it to top-up
+      // grids; a release after griddepcontrol.wait: the previous launch's main
+      // grid is complete and its results visible to whoever acquires this
+      if (b == 0) asm volatile("red.release.gpu.global.max.u32 [%0], %1;" ::"l"(&d->ctl->cur), "r"(d->req_idx) : "memory");
       S->hint_live = live;
       S->hint_alive = a;
     }
     const uint32_t launch_idx = d->launch_idx;
     // a dynamic total is the predecessor's output: read it after the wait
+    auto wait_prev = [&] {
+      if (cfg & kCfgWaitPrev) wait_complete(d - 1);   // not in stream order with it
+      else wait_topups(d - 1);                         // its main grid completed
+    };
     if constexpr (has_dynamic_total<T>::value) {
       if (topped_prev) {
-        wait_complete(d - 1);
+        wait_prev();
         topped_prev = 0;
       }
     }
     const uint32_t total = vg_total<T>(args, d, launch_idx);
-    // RESOLVE: every CTA publishes the total (the same value: a
-    // dynamic total is final once the predecessor launch completed).  Top-up
-    // CTAs may serve a launch before its main grid is resident -- when they
-    // fill the SMs the main grid waits for them -- so completion of a launch
-    // (wait_complete) must never depend on one particular CTA of the main grid
-    if (kResolve || blockIdx.x == 0) d->total_seen = total;
+    // Publish the total.  A static total: CTA 0 of either grid (the waiters
+    // of wait_topups follow the main grid, so its CTA 0 has run).  A dynamic
+    // total under RESOLVE: every CTA (the same value: it is final once the
+    // predecessor launch completed; an early grid's waiter must not depend on
+    // one particular CTA)
+    if ((kResolve && has_dynamic_total<T>::value) || blockIdx.x == 0) d->total_seen = total;
     S->chunk = chunk;
     S->have_nxt = 0;
     S->long_vg = 0;
@@ -494,14 +572,14 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     S->spread = has_spread<T>::value ? spread_factor(total) : 0u;
     S->prefetch_window = 2u * chunk * gridDim.x;
     S->template set_cur<has_spread<T>::value>(0, b);
-    if (topped_prev) wait_complete(d - 1);
+    if (topped_prev) wait_prev();
     if (cfg & kCfgStamps) red_min_u64(&d->t_first, globaltimer());
   }
   __syncthreads();
   // thread 0: the prefetched queue word and live quota stay in registers
   // across the body (a shared-memory store would wait for the atomic)
   unsigned long long r_v = 0;
-  uint32_t r_live = 0;
+  uint32_t r_live = 0, r_top = 1;
   for (uint32_t k = 0;; k ^= 1u) {
     const SchedState::Cur c = S->cur[k];
     if (c.vg >= S->total) break;                 // RUN_TERMINATE
@@ -514,7 +592,10 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
         // that idle time dwarfs one queue round trip) dequeue just in time
         // once fewer than two waves of VGs remain
         r_v = dequeue<kResolve>(d, S);
-        if (kResolve) r_live = (d->governed && !(cfg & kAblNoLive)) ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
+        if (kResolve) {
+          r_live = (d->governed && !(cfg & kAblNoLive)) ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
+          r_top = ld_relaxed(&d->topped);
+        }
         S->have_nxt = 1;
       }
       S->t0 = globaltimer();
@@ -535,7 +616,10 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
       } else {                                   // publish the prefetched chunk
         if (!S->have_nxt) {                      // tail: just in time
           r_v = dequeue<kResolve>(d, S);
-          if (kResolve) r_live = (d->governed && !(cfg & kAblNoLive)) ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
+          if (kResolve) {
+            r_live = (d->governed && !(cfg & kAblNoLive)) ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
+            r_top = ld_relaxed(&d->topped);
+          }
         }
         uint32_t nxt = kTerminate;
         if (r_v != kEvicted) {
@@ -543,6 +627,7 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
           if (kResolve) {
             S->hint_alive = qa_alive(r_v);   // admitted CTAs at our dequeue (incl. us)
             S->hint_live = r_live;
+            S->top_seen = r_top != 0u;
           }
         }
         S->end = nxt < S->total ? min(nxt + S->chunk, S->total) : nxt;
@@ -596,13 +681,14 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
   for (uint32_t l = s_l; l < sticky; ++l) {
     Desc* dl = d + l;
     if (threadIdx.x == 0) {
-      if (dl->has_prev) wait_complete(dl - 1);  // launch l's inputs are complete
+      if (dl->has_prev) wait_hybrid(dl - 1, dl->req_idx);  // launch l's inputs are complete
       atomicExch(&dl->topped, 1u);
+      atomicAdd(&dl->tu_alive, 1u);   // before the admission atomic (wait_topups)
       fence_acq_rel();
     }
     __syncthreads();
     // (the predecessor wait above already ran: no kCfgHasPrev)
-    const uint32_t cfg = dl->chunk | kCfgResolve | ((dl->flags & kFlagStamps) ? kCfgStamps : 0u);
+    const uint32_t cfg = dl->chunk | kCfgResolve | kCfgTopup | ((dl->flags & kFlagStamps) ? kCfgStamps : 0u);
     serve<T, true>(args, dl, smem, &S, cfg, blockIdx.x | 0x80000000u);
     __syncthreads();
     // a top-up CTA that was evicted (shrink) or admitted over the live quota

@@ -99,6 +99,10 @@ struct Request {
   // RESOLVE: one event after every top-up grid.  The request's descriptors
   // may only be released (and reused) once its sticky top-up CTAs retired.
   std::vector<cudaEvent_t> ev_topups;
+  // ACCEL_DEBUG: (tag, quota, event) of each re-solve -- 'L' after the live-quota
+  // write on the ctl stream, 'T' on the top-up stream just before a growth grid
+  struct DbgEv { char tag; uint32_t q; cudaEvent_t ev; };
+  std::vector<DbgEv> dbg;
   uint32_t slot = 0, n_desc = 0;
   uint32_t* cov = nullptr;
   uint64_t cov_elems = 0;
@@ -155,7 +159,7 @@ struct DescHost {
   uint32_t pad1[30];
   // line 2
   unsigned long long t_first, t_last;
-  uint32_t total_seen, ctas_started, pad_alive, max_alive, topped, admit_fail, evicted, last_live, pad_adm, draining, pad2[18];
+  uint32_t total_seen, ctas_started, tu_alive, max_alive, topped, admit_fail, evicted, last_live, pad_adm, draining, pad2[18];
 };
 static_assert(sizeof(DescHost) == accel::kDescBytes, "host view of the descriptor");
 
@@ -200,7 +204,8 @@ struct accel_ctx {
   std::thread monitor;
   std::atomic<bool> stop{false};
   uint64_t monitor_solves = 0;
-  uint32_t ablate = 0;   // env ACCEL_ABLATE: measurement-only cfg bits (dispatch.cuh kAbl*)
+  uint32_t ablate = 0;
+  std::chrono::steady_clock::time_point t_init = std::chrono::steady_clock::now();   // ACCEL_DEBUG stamps   // env ACCEL_ABLATE: measurement-only cfg bits (dispatch.cuh kAbl*)
   bool pdl = true;       // programmatic dependent launch between a request's launches (env ACCEL_PDL=0: off)
   std::vector<uint8_t> slot_used;
   std::map<uint64_t, std::unique_ptr<Request>> reqs;
@@ -253,6 +258,7 @@ struct accel_ctx {
 namespace {
 
 bool debug_on();
+double host_us(const accel_ctx* ctx);
 
 int refresh_done(accel_ctx* ctx, Request* r) {
   if (r->done) return ACCEL_OK;
@@ -318,6 +324,14 @@ int fetch_result(accel_ctx* ctx, Request* r) {
       }
     r->cov_ok = ok ? 1 : 0;
   }
+  for (const Request::DbgEv& x : r->dbg) {
+    float ms = -1.f;
+    cudaEventElapsedTime(&ms, r->ev_arrival, x.ev);
+    std::fprintf(stderr, "[accel] req %llu tenant %d re-solve %c q=%u at +%.1f us after arrival\n",
+                 (unsigned long long)r->id, r->tenant, x.tag, x.q, 1e3f * ms);
+    cudaEventDestroy(x.ev);
+  }
+  r->dbg.clear();
   r->fetched = true;
   return ACCEL_OK;
 }
@@ -429,8 +443,10 @@ int enqueue_next(accel_ctx* ctx, Request* r, bool* more) {
     accel::Desc* d = ctx->desc_ptr(r->slot + st.first + l);
     // accel_persistent cfg word (dispatch.cuh): chunk | kCfgResolve | kCfgStamps
     // | kCfgHasPrev (a request-relative launch precedes this one) | kCfgStaticFirst
+    // | kCfgAccount (RESOLVE, a request with an early main grid: its CTAs keep
+    // the fenced alive decrement the early grid's wait_complete counts on)
     uint32_t cfg = (k.chunk & 0xffffu) | (resolve ? (1u << 16) : 0u) | (1u << 17) | (li > 0 ? (1u << 18) : 0u) |
-                   (1u << 19) | ctx->ablate;
+                   (1u << 19) | (resolve && r->early_main ? (1u << 21) : 0u) | ctx->ablate;
     void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &cfg};
     const dim3 grid = shared ? dim3(st.quota, 1, 1) : dim3(st.grid.x, st.grid.y, st.grid.z);
     const void* fn = shared ? (resolve ? k.prfn : k.pfn) : k.nfn;
@@ -600,8 +616,18 @@ int apply_quota(accel_ctx* ctx, Request* r, uint32_t q) {
   // both the live-quota write and a growth grid must follow the request's
   // descriptor init (which writes live_init and resets the queue words): a
   // re-solve may come while the tenant stream is still copying its inputs
+  const double t_a = debug_on() ? host_us(ctx) : 0.0;
   CK(ctx, cudaStreamWaitEvent(ctx->ctl, r->ev_init, 0));
+  const double t_b = debug_on() ? host_us(ctx) : 0.0;
   CK(ctx, cudaMemcpyAsync(ctx->ctl_pool + (size_t)r->slot * kCtlBytes /* Ctl::live */, h, sizeof(uint32_t), cudaMemcpyHostToDevice, ctx->ctl));
+  if (debug_on()) {
+    cudaEvent_t ev;
+    CK(ctx, cudaEventCreate(&ev));
+    CK(ctx, cudaEventRecord(ev, ctx->ctl));
+    r->dbg.push_back({'L', q, ev});
+  }
+  const double t_c = debug_on() ? host_us(ctx) : 0.0;
+  double t_d = t_c, t_e = t_c;
   // (no growth grids for an early main step: they would wait beside it for
   // the earlier steps and could hold the SMs those need)
   if (q > r->provisioned && !r->early_main) {
@@ -612,13 +638,24 @@ int apply_quota(accel_ctx* ctx, Request* r, uint32_t q) {
     void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &sticky};
     cudaStream_t ts = ctx->pick_topup_stream();
     CK(ctx, cudaStreamWaitEvent(ts, r->ev_init, 0));
+    if (debug_on()) {
+      cudaEvent_t ev;
+      CK(ctx, cudaEventCreate(&ev));
+      CK(ctx, cudaEventRecord(ev, ts));
+      r->dbg.push_back({'T', q - r->provisioned, ev});
+    }
+    t_d = debug_on() ? host_us(ctx) : 0.0;
     CK(ctx, cudaLaunchKernel(k.tfn, dim3(q - r->provisioned, 1, 1), k.block, params, k.dyn_smem, ts));
+    t_e = debug_on() ? host_us(ctx) : 0.0;
     cudaEvent_t ev;
     CK(ctx, ctx->get_event(&ev));
     r->ev_topups.push_back(ev);
     CK(ctx, cudaEventRecord(ev, ts));
     r->provisioned = q;
   }
+  if (debug_on())
+    std::fprintf(stderr, "[accel] apply_quota us: wait %.1f memcpy %.1f prep %.1f launch %.1f rest %.1f\n", t_b - t_a,
+                 t_c - t_b, t_d - t_c, t_e - t_d, host_us(ctx) - t_e);
   // the CTAs a shrink evicts leave the running launch: a later growth must top up again
   if (q < r->live) r->provisioned = std::min(r->provisioned, q);
   r->live = q;
@@ -690,6 +727,10 @@ int assign_quotas(accel_ctx* ctx, std::vector<std::unique_ptr<Request>>& fresh) 
 
 // Host monitor (RESOLVE): detects departures without host synchronisation by
 // polling the requests' completion events, and re-solves the survivors.
+double host_us(const accel_ctx* ctx) {
+  return std::chrono::duration<double, std::micro>(std::chrono::steady_clock::now() - ctx->t_init).count();
+}
+
 void monitor_loop(accel_ctx* ctx) {
   cudaSetDevice(ctx->cfg.device);
   bool busy = false;
@@ -712,10 +753,12 @@ void monitor_loop(accel_ctx* ctx) {
       }
     }
     busy = running;
-    if (departed && debug_on()) std::fprintf(stderr, "[accel] monitor: departure (running=%d)\n", (int)running);
+    if (departed && debug_on()) std::fprintf(stderr, "[accel] monitor: departure (running=%d) at host %.1f us\n",
+                                             (int)running, host_us(ctx));
     if (departed && running) {
       std::vector<std::unique_ptr<Request>> none;
       assign_quotas(ctx, none);
+      if (debug_on()) std::fprintf(stderr, "[accel] monitor: re-solved at host %.1f us\n", host_us(ctx));
     }
   }
 }
@@ -966,7 +1009,10 @@ int accel_kernel_info_get(accel_ctx* ctx, int32_t kernel_id, accel_kernel_info* 
 int accel_submit_group(accel_ctx* ctx, uint32_t n, const accel_request* rs, uint64_t* ids) {
   if (!ctx || (n && (!rs || !ids))) return ACCEL_EINVAL;
   std::lock_guard<std::mutex> g(ctx->mu);
-  return submit_locked(ctx, n, rs, ids);
+  if (debug_on()) std::fprintf(stderr, "[accel] submit %u requests at host %.1f us\n", n, host_us(ctx));
+  const int rc = submit_locked(ctx, n, rs, ids);
+  if (debug_on()) std::fprintf(stderr, "[accel] submit done at host %.1f us\n", host_us(ctx));
+  return rc;
 }
 
 int accel_submit(accel_ctx* ctx, const accel_request* r, uint64_t* id) {
@@ -1003,10 +1049,11 @@ void dump_stuck(accel_ctx* ctx, const std::vector<uint64_t>& ids) {
     for (uint32_t l = 0; l < r->n_desc; ++l) {
       const DescHost* d = reinterpret_cast<const DescHost*>(h.data() + (size_t)l * kDescBytes);
       const uint32_t next = (uint32_t)d->qa, alive = (uint32_t)(d->qa >> 32);
-      if (d->total_seen != 0xffffffffu && next >= d->total_seen && alive == 0 && d->draining == 0) continue;
-      std::fprintf(stderr, "[accel]   launch %u: total %u seen %u next %u alive %u draining %u topped %u started %u "
-                           "refused %u evicted %u\n", l, d->total, d->total_seen, next, alive, d->draining, d->topped,
-                   d->ctas_started, d->admit_fail, d->evicted);
+      // (main-grid CTAs retire without decrementing `alive`: dispatch.cuh)
+      if (d->total_seen != 0xffffffffu && next >= d->total_seen && d->tu_alive == 0 && d->draining == 0) continue;
+      std::fprintf(stderr, "[accel]   launch %u: total %u seen %u next %u alive %u tu_alive %u draining %u topped %u "
+                           "started %u refused %u evicted %u\n", l, d->total, d->total_seen, next, alive, d->tu_alive,
+                   d->draining, d->topped, d->ctas_started, d->admit_fail, d->evicted);
     }
   }
   cudaStreamDestroy(st);

@@ -59,6 +59,7 @@ __global__ void desc_init_kernel(const InitParams p, uint32_t n_desc) {
   d->admit_fail = 0;
   d->evicted = 0;
   d->draining = 0;
+  d->tu_alive = 0;
   d->last_live = 0;
   d->topped = 0;
   d->req_idx = i;
@@ -66,10 +67,10 @@ __global__ void desc_init_kernel(const InitParams p, uint32_t n_desc) {
   d->qa = st.qa0;
 }
 
-// Request completion: wait until the last launch completed if another grid
-// (a RESOLVE top-up) may still be serving it.
+// Request completion: the last launch's main grid precedes this kernel in
+// stream order; wait for its top-up CTAs if a RESOLVE top-up grid joined it.
 __global__ void join_kernel(const Desc* last) {
-  if (threadIdx.x == 0 && ld_volatile(&last->topped)) wait_complete(last);
+  if (threadIdx.x == 0 && ld_volatile(&last->topped)) wait_topups(last);
 }
 
 cudaError_t launch_join(const Desc* last, cudaStream_t s) {
