@@ -158,6 +158,13 @@ __device__ __forceinline__ unsigned long long globaltimer() {
   asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
   return t;
 }
+// A persistent grid lets its successor launch only when its CTAs reach their
+// last VG (serve): a successor released at CTA start holds SM slots for the
+// whole launch -- waiting in griddepcontrol.wait -- and takes every slot a
+// co-runner frees in the meantime (measured: bfs's level grids waited 100-240
+// us each for slots behind the stencil's pre-launched sweeps in C2).
+__device__ __forceinline__ void pdl_wait() { asm volatile("griddepcontrol.wait;" ::: "memory"); }
+__device__ __forceinline__ void pdl_release() { asm volatile("griddepcontrol.launch_dependents;" ::: "memory"); }
 __device__ __forceinline__ uint32_t smid() {
   uint32_t v;
   asm volatile("mov.u32 %0, %%smid;" : "=r"(v));
@@ -387,6 +394,7 @@ struct SchedState {
   uint32_t hint_live, hint_alive;
   uint8_t have_nxt, admitted, draining;
   uint8_t top_seen;    // RESOLVE: the launch was topped at this CTA's last dequeue
+  uint8_t released;    // griddepcontrol.launch_dependents issued
   uint8_t over;        // RESOLVE: admitted over the live quota -> leave at the next dequeue
   uint8_t long_vg;     // the last VG ran longer than kLongVgNs
   template <bool kSpread>
@@ -488,6 +496,7 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     S->draining = 0;
     S->over = 0;
     S->top_seen = 1;   // (conservative until the first dynamic dequeue)
+    S->released = 0;
     // Static first chunk (main grids): measured, the first dequeue of 740
     // CTAs on one queue word serialised in L2 and spread the CTAs' first VG
     // starts over 6 us of a 30-us stencil launch (scripts/vg_trace.py)
@@ -516,6 +525,13 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
         // evicts at the next dequeue
         b = blockIdx.x * chunk;
         a = gridDim.x;
+        // CTA 0 holds the launch's first ticket: it announces the launch to
+        // top-up grids, a release after griddepcontrol.wait (the previous
+        // launch's main grid is complete and its results visible to whoever
+        // acquires this).  Issued before this thread's first store or
+        // reduction, so the release waits for nothing outstanding
+        if (blockIdx.x == 0)
+          asm volatile("red.release.gpu.global.max.u32 [%0], %1;" ::"l"(&d->ctl->cur), "r"(d->req_idx) : "memory");
         if (blockIdx.x == 0 && !(cfg & kAblNoStats))
           asm volatile("red.relaxed.gpu.global.max.u32 [%0], %1;" ::"l"(&d->max_alive), "r"(a) : "memory");
       } else {
@@ -530,10 +546,10 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
           d->last_live = live;
         }
       }
-      // the CTA holding the launch's first ticket announces it to top-up
-      // grids; a release after griddepcontrol.wait: the previous launch's main
-      // grid is complete and its results visible to whoever acquires this
-      if (b == 0) asm volatile("red.release.gpu.global.max.u32 [%0], %1;" ::"l"(&d->ctl->cur), "r"(d->req_idx) : "memory");
+      // (a queue-admitted CTA never holds ticket 0 under static first chunks;
+      // without them the CTA that does announces the launch, as above)
+      if (!stat && b == 0)
+        asm volatile("red.release.gpu.global.max.u32 [%0], %1;" ::"l"(&d->ctl->cur), "r"(d->req_idx) : "memory");
       S->hint_live = live;
       S->hint_alive = a;
     }
@@ -631,6 +647,12 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
           }
         }
         S->end = nxt < S->total ? min(nxt + S->chunk, S->total) : nxt;
+        // this CTA's last chunk (the queue will be dry at its next dequeue,
+        // or is already): let the request's next launch be scheduled
+        if (!S->released && (nxt >= S->total || S->total - nxt <= S->chunk * gridDim.x)) {
+          pdl_release();
+          S->released = 1;
+        }
         S->template set_cur<has_spread<T>::value>(k ^ 1u, nxt);
         S->have_nxt = 0;
       }
@@ -652,6 +674,7 @@ __device__ __forceinline__ void pdl_enter() {
   asm volatile("griddepcontrol.wait;" ::: "memory");
 }
 
+
 // -------------------------------------------------------------------------
 // The scheduling kernel: grid = quota (1-D), block = the original block;
 // serves launch d.  cfg = chunk | kCfg* flags.  kResolve = RESOLVE policy.
@@ -660,7 +683,7 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
     accel_persistent(const __grid_constant__ typename T::Args args, Desc* __restrict__ d, uint32_t cfg) {
   extern __shared__ __align__(128) char smem[];
   __shared__ SchedState S;
-  pdl_enter();
+  pdl_wait();
   serve<T, kResolve>(args, d, smem, &S, cfg, blockIdx.x);
 }
 
