@@ -30,13 +30,15 @@ def main():
     ap.add_argument("--tenants", default=",".join(TENANTS))
     ap.add_argument("--reps", type=int, default=3)
     ap.add_argument("--out", default=None)
+    ap.add_argument("--fracs", default=None, help="comma-separated device fractions (default: the full list)")
     a = ap.parse_args()
+    fracs = [float(x) for x in a.fracs.split(",")] if a.fracs else FRACS
     sms = torch.cuda.get_device_properties(0).multi_processor_count
     flush = torch.empty(64 * 1024 * 1024, dtype=torch.float32, device="cuda")
     tenants = a.tenants.split(",")
     inputs = {t: synth.preset(t, "default", seed=11) for t in tenants}
     prof = {t: {} for t in tenants}
-    for f in FRACS:
+    for f in fracs:
         s = max(1, round(f * sms))
         acc = Accel(0, mode=abi.MODE_SHARED, policy=abi.POLICY_STATIC, caps=abi.accel_caps(s, 0, 0, 0, 0))
         for t in tenants:
@@ -53,8 +55,8 @@ def main():
             prof[t][f] = {"ms": statistics.median(el[1:]), "quota": q, "sms": s}
             print(t, f, round(prof[t][f]["ms"], 4), q, flush=True)
         acc.close()
-    out = {"sms": sms, "fracs": FRACS,
-           "profile": {t: {"ms": [prof[t][f]["ms"] for f in FRACS], "quota": [prof[t][f]["quota"] for f in FRACS]}
+    out = {"sms": sms, "fracs": fracs,
+           "profile": {t: {"ms": [prof[t][f]["ms"] for f in fracs], "quota": [prof[t][f]["quota"] for f in fracs]}
                        for t in tenants}}
     print(json.dumps(out))
     if a.out:
