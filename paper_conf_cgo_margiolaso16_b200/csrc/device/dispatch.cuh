@@ -41,15 +41,19 @@
 // TOP-UP CTAs to be done: a top-up CTA counts itself in `tu_alive` before it
 // joins a launch and leaves it with a release fence + decrement
 // (wait_topups).  A top-up CTA is in no stream order with the main grids:
-// before it serves launch l+1 it needs launch l complete (wait_hybrid).  Main
-// CTAs that saw the launch `topped` at their last dequeue retire with a
-// release fence and the `alive` decrement, so a topped launch completes as
-// soon as its last CTA leaves (alive == 0); a main CTA of a launch no top-up
-// had joined retires with no fence and no atomic -- the single-tenant case --
-// and a top-up that joins such a launch late falls back to waiting until
-// launch l+1's main grid has STARTED (ctl->cur, a release by the CTA holding
-// l+1's first ticket after its griddepcontrol.wait: l's main grid is then
-// complete) and l's top-ups are done.  An early main grid (R-place-3,
+// before it serves launch l+1 it needs launch l complete (wait_hybrid).  Once
+// the monitor grows a request it sets ctl->grown (with the live quota, before
+// the first top-up grid); a main CTA that saw `grown` at its last dequeue
+// retires with a release fence and the `alive` decrement, so such a launch
+// completes as soon as its last CTA leaves (alive == 0).  A request that was
+// never grown -- always, alone -- retires its main CTAs with no fence and no
+// atomic.  For the launch that was running when the request grew, whose main
+// CTAs may not account, a top-up falls back to waiting until launch l+1's
+// main grid has STARTED (ctl->cur, a release by the CTA holding l+1's first
+// ticket after its griddepcontrol.wait: l's main grid is then complete) and
+// l's top-ups are done; that wait needs a free slot for l+1's CTA 0, so it is
+// bounded (kGiveUpNs) and a top-up that gives up leaves the request (always
+// safe: top-up CTAs are optional capacity).  An early main grid (R-place-3,
 // launched ahead on a side stream) waits for its predecessor's main CTAs too:
 // that request's launches carry kCfgAccount (every main CTA accounts).
 #pragma once
@@ -69,9 +73,12 @@ namespace accel {
 // red.max on it queued every CTA's live-quota load behind it in the L2 slice
 // (RESOLVE single-tenant overhead 16-21 % -> 10-11 % without it).
 struct alignas(128) Ctl {
-  // ---- line 0
+  // ---- line 0 (live and grown are read together, one 64-bit load)
   uint32_t live;      // live quota (RESOLVE)
-  uint32_t pad1[31];
+  uint32_t grown;     // the monitor has launched a top-up grid for this request
+                      // (written with `live`, before the grid): main CTAs account
+  uint32_t lost;      // top-up CTAs that gave up waiting for a launch (diagnostic)
+  uint32_t pad1[29];
   // ---- line 1
   uint32_t cur;       // highest request-relative launch index started (one red per launch)
   uint32_t pad2[31];
@@ -186,6 +193,13 @@ __device__ __forceinline__ uint32_t ld_relaxed(const uint32_t* p) {
   return v;
 }
 
+// {live, grown} of a Ctl line 0 in one load (live in the low half)
+__device__ __forceinline__ unsigned long long ld_relaxed_u64(const void* p) {
+  unsigned long long v;
+  asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+  return v;
+}
+
 __device__ __forceinline__ uint32_t ld_volatile(const uint32_t* p) {
   uint32_t v;
   asm volatile("ld.volatile.global.u32 %0, [%1];" : "=r"(v) : "l"(p));
@@ -296,9 +310,12 @@ __device__ __forceinline__ void wait_complete(const Desc* p) {
 
 // Top-up CTA: wait until launch p (the predecessor of request launch
 // `next_idx`) is complete -- every admitted CTA left (alive == 0: all of p's
-// main CTAs accounted because p was topped), or p's successor main grid has
-// started (p's main grid done) and p's own top-ups are done.
-__device__ __forceinline__ void wait_hybrid(const Desc* p, uint32_t next_idx) {
+// main CTAs accounted), or p's successor main grid has started (p's main grid
+// done) and p's own top-ups are done.  False if neither happened within
+// kGiveUpNs (the successor's CTA 0 found no slot): the caller leaves.
+constexpr unsigned long long kGiveUpNs = 500000;
+__device__ __forceinline__ bool wait_hybrid(const Desc* p, uint32_t next_idx) {
+  const unsigned long long t0 = globaltimer();
   for (;;) {
     const uint32_t tot = ld_volatile(&p->total_seen);
     const unsigned long long v = ld_volatile_u64(&p->qa);
@@ -312,10 +329,12 @@ __device__ __forceinline__ void wait_hybrid(const Desc* p, uint32_t next_idx) {
         if (ld_volatile(&p->tu_alive) == 0 && ld_volatile(&p->draining) == 0) break;
       }
     }
+    if (globaltimer() - t0 > kGiveUpNs) return false;
     __nanosleep(256);
   }
   fence_acq_rel();
   asm volatile("fence.proxy.async.global;" ::: "memory");
+  return true;
 }
 
 // Launch p's main grid is known complete (stream order, or ctl->cur past it):
@@ -393,7 +412,7 @@ struct SchedState {
   // latency in front of the queue atomic
   uint32_t hint_live, hint_alive;
   uint8_t have_nxt, admitted, draining;
-  uint8_t top_seen;    // RESOLVE: the launch was topped at this CTA's last dequeue
+  uint8_t top_seen;    // RESOLVE: the request was grown at this CTA's last dequeue
   uint8_t released;    // griddepcontrol.launch_dependents issued
   uint8_t over;        // RESOLVE: admitted over the live quota -> leave at the next dequeue
   uint8_t long_vg;     // the last VG ran longer than kLongVgNs
@@ -594,8 +613,7 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
   __syncthreads();
   // thread 0: the prefetched queue word and live quota stay in registers
   // across the body (a shared-memory store would wait for the atomic)
-  unsigned long long r_v = 0;
-  uint32_t r_live = 0, r_top = 1;
+  unsigned long long r_v = 0, r_ctl = 0;
   for (uint32_t k = 0;; k ^= 1u) {
     const SchedState::Cur c = S->cur[k];
     if (c.vg >= S->total) break;                 // RUN_TERMINATE
@@ -608,10 +626,7 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
         // that idle time dwarfs one queue round trip) dequeue just in time
         // once fewer than two waves of VGs remain
         r_v = dequeue<kResolve>(d, S);
-        if (kResolve) {
-          r_live = (d->governed && !(cfg & kAblNoLive)) ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
-          r_top = ld_relaxed(&d->topped);
-        }
+        if (kResolve) r_ctl = ld_relaxed_u64(&d->ctl->live);   // {live, grown}
         S->have_nxt = 1;
       }
       S->t0 = globaltimer();
@@ -632,18 +647,16 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
       } else {                                   // publish the prefetched chunk
         if (!S->have_nxt) {                      // tail: just in time
           r_v = dequeue<kResolve>(d, S);
-          if (kResolve) {
-            r_live = (d->governed && !(cfg & kAblNoLive)) ? ld_relaxed(&d->ctl->live) : 0xffffffffu;
-            r_top = ld_relaxed(&d->topped);
-          }
+          if (kResolve) r_ctl = ld_relaxed_u64(&d->ctl->live);
         }
         uint32_t nxt = kTerminate;
         if (r_v != kEvicted) {
           nxt = qa_next(r_v);
           if (kResolve) {
             S->hint_alive = qa_alive(r_v);   // admitted CTAs at our dequeue (incl. us)
-            S->hint_live = r_live;
-            S->top_seen = r_top != 0u;
+            // the live quota governs the request's main step only
+            S->hint_live = (d->governed && !(cfg & kAblNoLive)) ? (uint32_t)r_ctl : 0xffffffffu;
+            S->top_seen = (r_ctl >> 32) != 0u;   // grown: this CTA accounts at retire
           }
         }
         S->end = nxt < S->total ? min(nxt + S->chunk, S->total) : nxt;
@@ -695,7 +708,7 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
     accel_topup(const __grid_constant__ typename T::Args args, Desc* __restrict__ d, uint32_t sticky) {
   extern __shared__ __align__(128) char smem[];
   __shared__ SchedState S;
-  __shared__ uint32_t s_l;
+  __shared__ uint32_t s_l, s_go;
   if (threadIdx.x == 0) {
     const uint32_t cur = ld_volatile(&d->ctl->cur);
     s_l = cur > d->req_idx ? cur - d->req_idx : 0u;
@@ -704,12 +717,19 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
   for (uint32_t l = s_l; l < sticky; ++l) {
     Desc* dl = d + l;
     if (threadIdx.x == 0) {
-      if (dl->has_prev) wait_hybrid(dl - 1, dl->req_idx);  // launch l's inputs are complete
-      atomicExch(&dl->topped, 1u);
-      atomicAdd(&dl->tu_alive, 1u);   // before the admission atomic (wait_topups)
-      fence_acq_rel();
+      s_go = 1u;
+      // launch l's inputs are complete (or the wait gave up: leave)
+      if (dl->has_prev && !wait_hybrid(dl - 1, dl->req_idx)) {
+        s_go = 0u;
+        red_add_u32(&dl->ctl->lost, 1u);
+      } else {
+        atomicExch(&dl->topped, 1u);
+        atomicAdd(&dl->tu_alive, 1u);   // before the admission atomic (wait_topups)
+        fence_acq_rel();
+      }
     }
     __syncthreads();
+    if (!s_go) return;
     // (the predecessor wait above already ran: no kCfgHasPrev)
     const uint32_t cfg = dl->chunk | kCfgResolve | kCfgTopup | ((dl->flags & kFlagStamps) ? kCfgStamps : 0u);
     serve<T, true>(args, dl, smem, &S, cfg, blockIdx.x | 0x80000000u);

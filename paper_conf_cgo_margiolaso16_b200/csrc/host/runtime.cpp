@@ -112,6 +112,7 @@ struct Request {
   size_t enq_step = 0;       // enqueue cursor (enqueue_next)
   uint32_t enq_launch = 0, enq_li = 0;
   bool early_main = false;   // R-place-3: main step launched ahead on a side stream
+  bool grown = false;        // RESOLVE: a top-up grid was launched (device Ctl::grown)
   uint32_t early_sms = 0;    // SMs its waiting grid may hold (released when done)
   cudaEvent_t ev_early = nullptr;  // recorded after that launch (the main stream waits for it)
   uint32_t live = 0;         // RESOLVE: current live quota of the main step
@@ -611,15 +612,27 @@ int apply_quota(accel_ctx* ctx, Request* r, uint32_t q) {
                  (unsigned long long)r->id, r->tenant, r->live, q, r->provisioned);
   if (q == r->live || r->ev_init == nullptr) return ACCEL_OK;
   if (cudaEventQuery(r->ev_done) == cudaSuccess) return ACCEL_OK;  // finished: nothing to grow
-  uint32_t* h = ctx->pinned_ring + (ctx->ring_pos++ % kRing);
-  *h = q;
+  // {live, grown} (Ctl line 0), one 8-byte copy; grown is set before the
+  // request's first top-up grid (that grid waits for this copy), so main CTAs
+  // that see it account at retire (dispatch.cuh "completion accounting")
+  const bool grow = q > r->provisioned && !r->early_main;
+  uint32_t* h = ctx->pinned_ring + 2 * (ctx->ring_pos++ % (kRing / 2));
+  h[0] = q;
+  h[1] = (r->grown || grow) ? 1u : 0u;
   // both the live-quota write and a growth grid must follow the request's
   // descriptor init (which writes live_init and resets the queue words): a
   // re-solve may come while the tenant stream is still copying its inputs
   const double t_a = debug_on() ? host_us(ctx) : 0.0;
   CK(ctx, cudaStreamWaitEvent(ctx->ctl, r->ev_init, 0));
   const double t_b = debug_on() ? host_us(ctx) : 0.0;
-  CK(ctx, cudaMemcpyAsync(ctx->ctl_pool + (size_t)r->slot * kCtlBytes /* Ctl::live */, h, sizeof(uint32_t), cudaMemcpyHostToDevice, ctx->ctl));
+  CK(ctx, cudaMemcpyAsync(ctx->ctl_pool + (size_t)r->slot * kCtlBytes /* Ctl::live, Ctl::grown */, h,
+                          2 * sizeof(uint32_t), cudaMemcpyHostToDevice, ctx->ctl));
+  cudaEvent_t ev_ctl = nullptr;
+  if (grow) {
+    CK(ctx, ctx->get_event(&ev_ctl));
+    CK(ctx, cudaEventRecord(ev_ctl, ctx->ctl));
+    r->ev_topups.push_back(ev_ctl);   // (recycled with the request's events)
+  }
   if (debug_on()) {
     cudaEvent_t ev;
     CK(ctx, cudaEventCreate(&ev));
@@ -630,7 +643,8 @@ int apply_quota(accel_ctx* ctx, Request* r, uint32_t q) {
   double t_d = t_c, t_e = t_c;
   // (no growth grids for an early main step: they would wait beside it for
   // the earlier steps and could hold the SMs those need)
-  if (q > r->provisioned && !r->early_main) {
+  if (grow) {
+    r->grown = true;
     const Step& st = r->steps[r->main_step];
     const Kernel& k = ctx->kernels[st.kid];
     accel::Desc* d = ctx->desc_ptr(r->slot + st.first);
@@ -638,6 +652,7 @@ int apply_quota(accel_ctx* ctx, Request* r, uint32_t q) {
     void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &sticky};
     cudaStream_t ts = ctx->pick_topup_stream();
     CK(ctx, cudaStreamWaitEvent(ts, r->ev_init, 0));
+    CK(ctx, cudaStreamWaitEvent(ts, ev_ctl, 0));   // Ctl::grown is set before any top-up CTA runs
     if (debug_on()) {
       cudaEvent_t ev;
       CK(ctx, cudaEventCreate(&ev));

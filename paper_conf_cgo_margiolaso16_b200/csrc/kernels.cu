@@ -31,6 +31,8 @@ __global__ void desc_init_kernel(const InitParams p, uint32_t n_desc) {
   const uint32_t i = blockIdx.x * blockDim.x + threadIdx.x;
   if (i == 0 && p.ctl != nullptr) {
     p.ctl->live = p.live_init;
+    p.ctl->grown = 0;
+    p.ctl->lost = 0;
     p.ctl->cur = 0;
   }
   if (i >= n_desc) return;

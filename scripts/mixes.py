@@ -211,8 +211,11 @@ def sampled(r: Runner, ta, reps, k, n, seed, repeat=False):
                 w = [max(1, round(16 * (ta[t] / tmax) ** ALPHA)) for t in names]
             runs = [mix_metrics(r.run(jobs, mode, pol, weights=w), [ta[t] for t in names]) for _ in range(reps)]
             res[name] = {kk: statistics.mean(x[kk] for x in runs) for kk in keys}
+            # per-tenant slowdowns T(s)/T(a) (which tenant sets U)
+            res[name]["s"] = [statistics.mean(x["ts_ms"][i] for x in runs) / ta[t] for i, t in enumerate(names)]
         mixes.append(res)
-        print(json.dumps({"mix": names, **{nm: {kk: round(v, 3) for kk, v in res[nm].items()} for nm, _, _ in MODES}}),
+        print(json.dumps({"mix": names, **{nm: {kk: (round(v, 3) if kk != "s" else [round(x, 3) for x in v])
+                                                 for kk, v in res[nm].items()} for nm, _, _ in MODES}}),
               flush=True)
     out = {}
     for name in SHARED:
