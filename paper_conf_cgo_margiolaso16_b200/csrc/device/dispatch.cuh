@@ -67,6 +67,24 @@
 
 namespace accel {
 
+// measurement-only compile-time switches (A/B builds; all 0 in the product)
+#ifndef ACCEL_XP_NOTOPPED
+#define ACCEL_XP_NOTOPPED 0
+#endif
+#ifndef ACCEL_XP_NOCUR
+#define ACCEL_XP_NOCUR 0
+#endif
+#ifndef ACCEL_XP_NOCTL
+#define ACCEL_XP_NOCTL 0
+#endif
+#ifndef ACCEL_XP_STRONGCTL
+#define ACCEL_XP_STRONGCTL 0
+#endif
+#ifndef ACCEL_XP_SAMPLECTL
+#define ACCEL_XP_SAMPLECTL 0
+#endif
+
+
 // Per-request control block (device memory), two 128-B lines: line 0 is
 // read at every admission and dequeue (the live quota), line 1 takes the
 // reductions.  Measured: with `cur` on the live quota's line, the per-CTA
@@ -193,11 +211,20 @@ __device__ __forceinline__ uint32_t ld_relaxed(const uint32_t* p) {
   return v;
 }
 
-// {live, grown} of a Ctl line 0 in one load (live in the low half)
-__device__ __forceinline__ unsigned long long ld_relaxed_u64(const void* p) {
+// {live, grown} of a Ctl line 0 in one load (live in the low half).  A weak
+// L2 load (.cg: no L1 copy that could go stale), not a strong one: a strong
+// load right behind the dequeue atomic measured 0.5 us per stencil launch
+// and 1.6 us per lbm launch; a view a few hundred ns old is all the
+// protocol needs (shrink at a later dequeue, accounting from `grown`, which
+// the host writes before any top-up CTA can run).
+__device__ __forceinline__ unsigned long long ld_ctl(const void* p) {
+#if ACCEL_XP_STRONGCTL
   unsigned long long v;
   asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
   return v;
+#else
+  return __ldcg(reinterpret_cast<const unsigned long long*>(p));
+#endif
 }
 
 __device__ __forceinline__ uint32_t ld_volatile(const uint32_t* p) {
@@ -406,6 +433,8 @@ struct SchedState {
   uint32_t* coverage;
   accel_vg_record* trace;
   const uint32_t* order;   // dequeue order of the launch (nullptr: linear / spread)
+  Ctl* ctl;                // RESOLVE: the request's control block (d->ctl)
+  uint32_t governed;       // RESOLVE: the live quota governs this launch
   unsigned long long t0;   // trace: start of the current VG
   // RESOLVE, thread 0: view of the live quota and the admitted count, loaded
   // right after each dequeue and used at the next one, so the check adds no
@@ -414,6 +443,17 @@ struct SchedState {
   uint8_t have_nxt, admitted, draining;
   uint8_t top_seen;    // RESOLVE: the request was grown at this CTA's last dequeue
   uint8_t released;    // griddepcontrol.launch_dependents issued
+  uint8_t ndq;         // RESOLVE: dequeues so far (ACCEL_XP_SAMPLECTL)
+  // RESOLVE: read the control line at this dequeue?  Always in the product;
+  // ACCEL_XP_SAMPLECTL (measurement): every 4th dequeue, every dequeue of a
+  // CTA whose VGs run long, and every dequeue in the launch's last two waves.
+  __device__ __forceinline__ bool ctl_due() {
+#if ACCEL_XP_SAMPLECTL
+    return long_vg || (ndq++ & 3u) == 0u || total - end <= 2u * chunk * gridDim.x;
+#else
+    return true;
+#endif
+  }
   uint8_t over;        // RESOLVE: admitted over the live quota -> leave at the next dequeue
   uint8_t long_vg;     // the last VG ran longer than kLongVgNs
   template <bool kSpread>
@@ -516,6 +556,7 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     S->over = 0;
     S->top_seen = 1;   // (conservative until the first dynamic dequeue)
     S->released = 0;
+    S->ndq = 0;
     // Static first chunk (main grids): measured, the first dequeue of 740
     // CTAs on one queue word serialised in L2 and spread the CTAs' first VG
     // starts over 6 us of a 30-us stencil launch (scripts/vg_trace.py)
@@ -531,7 +572,7 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
       // pays no serial round trip for it
       topped_prev =
           (cfg & kCfgWaitPrev) ? 1u
-          : ((cfg & kCfgHasPrev) && !(cfg & kAblNoTop)) ? ld_volatile(&(d - 1)->topped) : 0u;
+          : ((cfg & kCfgHasPrev) && !(cfg & kAblNoTop) && !ACCEL_XP_NOTOPPED) ? ld_volatile(&(d - 1)->topped) : 0u;
       // admission and first dequeue in one atomic; an arrival over the live
       // quota runs the chunk it got and leaves at its next dequeue
       // (a static-first CTA reads the live quota after its first dynamic
@@ -549,7 +590,7 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
         // launch's main grid is complete and its results visible to whoever
         // acquires this).  Issued before this thread's first store or
         // reduction, so the release waits for nothing outstanding
-        if (blockIdx.x == 0)
+        if (blockIdx.x == 0 && !ACCEL_XP_NOCUR)
           asm volatile("red.release.gpu.global.max.u32 [%0], %1;" ::"l"(&d->ctl->cur), "r"(d->req_idx) : "memory");
         if (blockIdx.x == 0 && !(cfg & kAblNoStats))
           asm volatile("red.relaxed.gpu.global.max.u32 [%0], %1;" ::"l"(&d->max_alive), "r"(a) : "memory");
@@ -604,6 +645,14 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     S->coverage = d->coverage;
     S->trace = d->trace;
     S->order = d->order;
+    // descriptor fields the dequeue loop needs, kept in shared memory: a
+    // descriptor load there is an L1 miss (and an L2 round trip in front of
+    // the dequeue atomic) whenever the tenant's body evicted the line --
+    // measured ~0.8 us per stencil launch under RESOLVE
+    if (kResolve) {
+      S->ctl = d->ctl;
+      S->governed = d->governed && !(cfg & kAblNoLive);
+    }
     S->spread = has_spread<T>::value ? spread_factor(total) : 0u;
     S->prefetch_window = 2u * chunk * gridDim.x;
     S->template set_cur<has_spread<T>::value>(0, b);
@@ -613,7 +662,7 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
   __syncthreads();
   // thread 0: the prefetched queue word and live quota stay in registers
   // across the body (a shared-memory store would wait for the atomic)
-  unsigned long long r_v = 0, r_ctl = 0;
+  unsigned long long r_v = 0, r_ctl = 0xffffffffull;   // (live = max, grown = 0 until loaded)
   for (uint32_t k = 0;; k ^= 1u) {
     const SchedState::Cur c = S->cur[k];
     if (c.vg >= S->total) break;                 // RUN_TERMINATE
@@ -625,8 +674,9 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
         // for up to one VG duration.  So kernels whose VGs run long (where
         // that idle time dwarfs one queue round trip) dequeue just in time
         // once fewer than two waves of VGs remain
+        // the control line ({live, grown}) is read beside every dequeue
+        if (kResolve && !ACCEL_XP_NOCTL && S->ctl_due()) r_ctl = ld_ctl(&S->ctl->live);
         r_v = dequeue<kResolve>(d, S);
-        if (kResolve) r_ctl = ld_relaxed_u64(&d->ctl->live);   // {live, grown}
         S->have_nxt = 1;
       }
       S->t0 = globaltimer();
@@ -646,8 +696,8 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
         S->template set_cur<has_spread<T>::value>(k ^ 1u, vg + 1);
       } else {                                   // publish the prefetched chunk
         if (!S->have_nxt) {                      // tail: just in time
+          if (kResolve && !ACCEL_XP_NOCTL && S->ctl_due()) r_ctl = ld_ctl(&S->ctl->live);
           r_v = dequeue<kResolve>(d, S);
-          if (kResolve) r_ctl = ld_relaxed_u64(&d->ctl->live);
         }
         uint32_t nxt = kTerminate;
         if (r_v != kEvicted) {
@@ -655,7 +705,7 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
           if (kResolve) {
             S->hint_alive = qa_alive(r_v);   // admitted CTAs at our dequeue (incl. us)
             // the live quota governs the request's main step only
-            S->hint_live = (d->governed && !(cfg & kAblNoLive)) ? (uint32_t)r_ctl : 0xffffffffu;
+            S->hint_live = S->governed ? (uint32_t)r_ctl : 0xffffffffu;
             S->top_seen = (r_ctl >> 32) != 0u;   // grown: this CTA accounts at retire
           }
         }

@@ -325,6 +325,19 @@ int fetch_result(accel_ctx* ctx, Request* r) {
       }
     r->cov_ok = ok ? 1 : 0;
   }
+  if (debug_on()) {
+    uint64_t ev = 0, af = 0, mx = 0, tu = 0;
+    for (uint32_t l = 0; l < r->n_desc; ++l) {
+      const DescHost* d = reinterpret_cast<const DescHost*>(r->desc_host.data() + (size_t)l * kDescBytes);
+      ev += d->evicted;
+      af += d->admit_fail;
+      mx = std::max<uint64_t>(mx, d->max_alive);
+      tu += d->topped;
+    }
+    std::fprintf(stderr, "[accel] req %llu tenant %d: %u launches, evicted %llu, refused %llu, max_alive %llu, topped %llu\n",
+                 (unsigned long long)r->id, r->tenant, r->n_desc, (unsigned long long)ev, (unsigned long long)af,
+                 (unsigned long long)mx, (unsigned long long)tu);
+  }
   for (const Request::DbgEv& x : r->dbg) {
     float ms = -1.f;
     cudaEventElapsedTime(&ms, r->ev_arrival, x.ev);
