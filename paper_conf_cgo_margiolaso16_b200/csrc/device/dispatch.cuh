@@ -80,6 +80,9 @@ namespace accel {
 #ifndef ACCEL_XP_STRONGCTL
 #define ACCEL_XP_STRONGCTL 0
 #endif
+#ifndef ACCEL_XP_PDL
+#define ACCEL_XP_PDL 1   // 0: release at CTA start, 1: at the last chunk, 2: at half the queue
+#endif
 #ifndef ACCEL_XP_SAMPLECTL
 #define ACCEL_XP_SAMPLECTL 0
 #endif
@@ -439,9 +442,7 @@ struct SchedState {
   // RESOLVE, thread 0: view of the live quota and the admitted count, loaded
   // right after each dequeue and used at the next one, so the check adds no
   // latency in front of the queue atomic
-  uint32_t hint_live, hint_alive;
   uint8_t have_nxt, admitted, draining;
-  uint8_t top_seen;    // RESOLVE: the request was grown at this CTA's last dequeue
   uint8_t released;    // griddepcontrol.launch_dependents issued
   uint8_t ndq;         // RESOLVE: dequeues so far (ACCEL_XP_SAMPLECTL)
   // RESOLVE: read the control line at this dequeue?  Always in the product;
@@ -514,19 +515,26 @@ __device__ __forceinline__ bool try_leave(Desc* d, SchedState* S) {
   return false;
 }
 
+// hint_alive / hint_live: this CTA's view from its previous dequeue (the
+// admitted count it returned, the live quota read beside it), in registers.
 template <bool kResolve>
-__device__ __forceinline__ unsigned long long dequeue(Desc* d, SchedState* S) {
-  if (kResolve && (S->over || S->hint_alive > S->hint_live) && try_leave(d, S))
+__device__ __forceinline__ unsigned long long dequeue(Desc* d, SchedState* S, uint32_t hint_alive,
+                                                      uint32_t hint_live) {
+  if (kResolve && (S->over || hint_alive > hint_live) && try_leave(d, S))
     return kEvicted;
   return atomicAdd(&d->qa, (unsigned long long)S->chunk);
 }
 
+// ctl_view: {live, grown} as read beside this CTA's last dequeue (~0 if it
+// never dequeued: it then accounts, conservatively)
 template <bool kResolve>
-__device__ __forceinline__ void retire(Desc* d, uint32_t cfg, const SchedState* S) {
+__device__ __forceinline__ void retire(Desc* d, uint32_t cfg, const SchedState* S, unsigned long long ctl_view) {
   if (kResolve) {
     // a main-grid CTA that ran until the queue was dry retires silently: its
-    // results reach its waiters through stream order (see the header)
-    if (S->admitted && ((cfg & (kCfgAccount | kCfgTopup)) || S->top_seen)) {
+    // results reach its waiters through stream order (see the header); once
+    // the request was grown, it accounts for the top-ups' sake
+    const bool grown = (ctl_view >> 32) != 0u;
+    if (S->admitted && ((cfg & (kCfgAccount | kCfgTopup)) || grown)) {
       if (!(cfg & kAblNoFence)) fence_acq_rel();  // this CTA's VG results before the alive decrement
       if (!(cfg & kAblNoDec)) atomicAdd(&d->qa, kAliveNeg);
     }
@@ -554,7 +562,6 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     S->admitted = 1;
     S->draining = 0;
     S->over = 0;
-    S->top_seen = 1;   // (conservative until the first dynamic dequeue)
     S->released = 0;
     S->ndq = 0;
     // Static first chunk (main grids): measured, the first dequeue of 740
@@ -610,8 +617,6 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
       // without them the CTA that does announces the launch, as above)
       if (!stat && b == 0)
         asm volatile("red.release.gpu.global.max.u32 [%0], %1;" ::"l"(&d->ctl->cur), "r"(d->req_idx) : "memory");
-      S->hint_live = live;
-      S->hint_alive = a;
     }
     const uint32_t launch_idx = d->launch_idx;
     // a dynamic total is the predecessor's output: read it after the wait
@@ -662,7 +667,15 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
   __syncthreads();
   // thread 0: the prefetched queue word and live quota stay in registers
   // across the body (a shared-memory store would wait for the atomic)
-  unsigned long long r_v = 0, r_ctl = 0xffffffffull;   // (live = max, grown = 0 until loaded)
+  // thread 0's view for the RESOLVE checks: the last queue word and control
+  // line {live, grown} (~0 until read: live = max, grown = conservative)
+  unsigned long long r_v = 0, r_ctl = ~0ull;
+  // RESOLVE hints from the previous dequeue (evaluated before r_v / r_ctl are
+  // overwritten; the live quota governs the request's main step only)
+  auto hints = [&](uint32_t* ha, uint32_t* hl) {
+    *ha = qa_alive(r_v);
+    *hl = S->governed ? (uint32_t)r_ctl : 0xffffffffu;
+  };
   for (uint32_t k = 0;; k ^= 1u) {
     const SchedState::Cur c = S->cur[k];
     if (c.vg >= S->total) break;                 // RUN_TERMINATE
@@ -675,8 +688,10 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
         // that idle time dwarfs one queue round trip) dequeue just in time
         // once fewer than two waves of VGs remain
         // the control line ({live, grown}) is read beside every dequeue
+        uint32_t ha = 0, hl = 0xffffffffu;
+        if (kResolve) hints(&ha, &hl);
         if (kResolve && !ACCEL_XP_NOCTL && S->ctl_due()) r_ctl = ld_ctl(&S->ctl->live);
-        r_v = dequeue<kResolve>(d, S);
+        r_v = dequeue<kResolve>(d, S, ha, hl);
         S->have_nxt = 1;
       }
       S->t0 = globaltimer();
@@ -696,23 +711,18 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
         S->template set_cur<has_spread<T>::value>(k ^ 1u, vg + 1);
       } else {                                   // publish the prefetched chunk
         if (!S->have_nxt) {                      // tail: just in time
+          uint32_t ha = 0, hl = 0xffffffffu;
+          if (kResolve) hints(&ha, &hl);
           if (kResolve && !ACCEL_XP_NOCTL && S->ctl_due()) r_ctl = ld_ctl(&S->ctl->live);
-          r_v = dequeue<kResolve>(d, S);
+          r_v = dequeue<kResolve>(d, S, ha, hl);
         }
-        uint32_t nxt = kTerminate;
-        if (r_v != kEvicted) {
-          nxt = qa_next(r_v);
-          if (kResolve) {
-            S->hint_alive = qa_alive(r_v);   // admitted CTAs at our dequeue (incl. us)
-            // the live quota governs the request's main step only
-            S->hint_live = S->governed ? (uint32_t)r_ctl : 0xffffffffu;
-            S->top_seen = (r_ctl >> 32) != 0u;   // grown: this CTA accounts at retire
-          }
-        }
+        const uint32_t nxt = r_v != kEvicted ? qa_next(r_v) : kTerminate;
         S->end = nxt < S->total ? min(nxt + S->chunk, S->total) : nxt;
         // this CTA's last chunk (the queue will be dry at its next dequeue,
         // or is already): let the request's next launch be scheduled
-        if (!S->released && (nxt >= S->total || S->total - nxt <= S->chunk * gridDim.x)) {
+        if (ACCEL_XP_PDL != 0 && !S->released &&
+            (nxt >= S->total ||
+             (ACCEL_XP_PDL == 1 ? S->total - nxt <= S->chunk * gridDim.x : 2u * nxt >= S->total))) {
           pdl_release();
           S->released = 1;
         }
@@ -722,7 +732,7 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     }
     __syncthreads();
   }
-  if (threadIdx.x == 0) retire<kResolve>(d, cfg, S);
+  if (threadIdx.x == 0) retire<kResolve>(d, cfg, S, r_ctl);
 }
 
 // Programmatic dependent launch (sm_90+): a request's launch l+1 is launched
@@ -746,6 +756,9 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
     accel_persistent(const __grid_constant__ typename T::Args args, Desc* __restrict__ d, uint32_t cfg) {
   extern __shared__ __align__(128) char smem[];
   __shared__ SchedState S;
+#if ACCEL_XP_PDL == 0
+  pdl_release();
+#endif
   pdl_wait();
   serve<T, kResolve>(args, d, smem, &S, cfg, blockIdx.x);
 }
