@@ -183,6 +183,25 @@ struct accel_ctx {
   // a growth grid is sticky (it follows its step's later launches), so a grid
   // queued behind another request's on the same stream would not start until
   // that one's step ends: take an idle top-up stream when there is one
+  // Coverage / trace buffers recycled by size: a cudaMalloc per submit stalls
+  // the submitting thread (and so the arrival of the next request) for 0.1-1 ms
+  std::multimap<size_t, void*> buf_pool;
+  cudaError_t buf_get(void** p, size_t bytes) {
+    auto it = buf_pool.find(bytes);
+    if (it != buf_pool.end()) {
+      *p = it->second;
+      buf_pool.erase(it);
+      return cudaSuccess;
+    }
+    return cudaMalloc(p, bytes);
+  }
+  void buf_put(void* p, size_t bytes) {
+    if (buf_pool.size() >= 64) {
+      cudaFree(p);
+      return;
+    }
+    buf_pool.emplace(bytes, p);
+  }
   cudaStream_t pick_topup_stream() {
     for (int i = 0; i < kTopupStreams; ++i) {
       const uint32_t k = (topup_rr + (uint32_t)i) % kTopupStreams;
@@ -814,8 +833,9 @@ int submit_locked(accel_ctx* ctx, uint32_t n, const accel_request* rs, uint64_t*
       return ctx->fail(ACCEL_ENOMEM, "descriptor pool exhausted (release finished requests)");
     }
     r->slot = (uint32_t)s;
-    if (r->cov_elems) CK(ctx, cudaMalloc(&r->cov, r->cov_elems * sizeof(uint32_t)));
-    if (r->trace_elems) CK(ctx, cudaMalloc(&r->trace, r->trace_elems * sizeof(accel_vg_record)));
+    if (r->cov_elems) CK(ctx, ctx->buf_get(reinterpret_cast<void**>(&r->cov), r->cov_elems * sizeof(uint32_t)));
+    if (r->trace_elems)
+      CK(ctx, ctx->buf_get(reinterpret_cast<void**>(&r->trace), r->trace_elems * sizeof(accel_vg_record)));
   }
   // SHARED: requests that arrive together are enqueued largest per-CTA
   // footprint first (dominant share of one SM, DESIGN.md R-place-1).  The
@@ -852,8 +872,8 @@ int submit_locked(accel_ctx* ctx, uint32_t n, const accel_request* rs, uint64_t*
 
 void release_request(accel_ctx* ctx, Request* r) {
   ctx->free_slots(r->slot, r->n_desc);
-  if (r->cov) cudaFree(r->cov);
-  if (r->trace) cudaFree(r->trace);
+  if (r->cov) ctx->buf_put(r->cov, r->cov_elems * sizeof(uint32_t));
+  if (r->trace) ctx->buf_put(r->trace, r->trace_elems * sizeof(accel_vg_record));
   if (r->ev_arrival) ctx->free_events.push_back(r->ev_arrival);
   if (r->ev_done) ctx->free_events.push_back(r->ev_done);
   if (r->ev_early) ctx->free_events.push_back(r->ev_early);
@@ -943,6 +963,7 @@ int accel_finalize(accel_ctx* ctx) {
   if (ctx->ctl) cudaStreamDestroy(ctx->ctl);
   if (ctx->ostream) cudaStreamDestroy(ctx->ostream);
   if (ctx->epoch) cudaEventDestroy(ctx->epoch);
+  for (auto& kv : ctx->buf_pool) cudaFree(kv.second);
   if (ctx->pool) cudaFree(ctx->pool);
   if (ctx->ctl_pool) cudaFree(ctx->ctl_pool);
   if (ctx->pinned_ring) cudaFreeHost(ctx->pinned_ring);
