@@ -46,7 +46,9 @@ typedef struct {
  * faces copy the input.  a0/buf0/buf1: DEVICE pointers to nx*ny*nz floats,
  * 16-B aligned, no padding required.
  * Kernel "stencil2" (same arguments, nx % 4 == 0): VG tile 128 x 16 x 8, two
- * rows per warp -- grid (ceil(nx/128), ceil(ny/16), ceil(nz/8)). */
+ * rows per warp -- grid (ceil(nx/128), ceil(ny/16), ceil(nz/8)).
+ * Kernel "stencil_z16" (same arguments, nx % 4 == 0): VG tile 128 x 8 x 16 --
+ * grid (ceil(nx/128), ceil(ny/8), ceil(nz/16)). */
 typedef struct {
   const float *a0;
   float *buf0;
@@ -72,6 +74,12 @@ typedef struct {
                                this DEVICE array instead of the parameters */
   const float *a0;          /* the input volume (kernel "stencil_bulk": 1-D
                                bulk copies need no tensor map) */
+  uint32_t *dbg;            /* diagnostic: non-NULL = DEVICE block; consumers
+                               compare every staged plane row with an L2 load
+                               of the same input (scripts/diag_tma_check.py):
+                               dbg[0] = mismatches, dbg[8 + 8k ..] = record k
+                               {launch, z, y, x, staged bits, L2 bits, sm,
+                               output-buffer bits} for k < 16 */
 } accel_stencil_tma_args;
 
 /* histo -- saturating histogram (Parboil histo main + final fused).

@@ -118,7 +118,7 @@ class accel_stencil_tma_args(C.Structure):
     # three 128-B CUtensorMaps first; the C struct is 64-B aligned, so its
     # size is rounded up to a multiple of 64 (trailing pad)
     _fields_ = [("tmaps", C.c_uint8 * 384), ("buf0", vp), ("buf1", vp), ("nx", u32), ("ny", u32), ("nz", u32),
-                ("c0", f32), ("c1", f32), ("l2hint", u32), ("gmaps", vp), ("a0", vp), ("_pad", C.c_uint8 * 8)]
+                ("c0", f32), ("c1", f32), ("l2hint", u32), ("gmaps", vp), ("a0", vp), ("dbg", vp)]
 
 
 class accel_histo_args(C.Structure):
@@ -164,6 +164,7 @@ accel_sgemm_tc1_args = accel_sgemm_tc_args
 accel_spmv_v4_args = accel_spmv_args
 accel_stencil_deep_args = accel_stencil_args
 accel_stencil2_args = accel_stencil_args
+accel_stencil_z16_args = accel_stencil_args
 accel_stencil_bulk_args = accel_stencil_tma_args
 accel_histo_wide_args = accel_histo_args
 

@@ -118,6 +118,7 @@ const Builtin kBuiltins[] = {
     {"stencil", &make_desc<Stencil>},
     {"stencil_x", &make_desc<StencilX>},
     {"stencil_deep", &make_desc<StencilDeep>},
+    {"stencil_z16", &make_desc<StencilZ16>},
     {"stencil2", &make_desc<Stencil2>},
     {"stencil_tma", &make_desc<StencilTma>},
     {"stencil_bulk", &make_desc<StencilBulk>},

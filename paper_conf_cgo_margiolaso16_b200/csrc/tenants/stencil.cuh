@@ -36,11 +36,13 @@ namespace accel {
 #endif
 // kDepth: planes in flight beyond z+1 ("stencil_deep": the whole 10-plane
 // tile in flight per VG -- more bytes in flight per CTA for a small share)
-template <bool kAligned, int kDepth = STENCIL_KD>
+// kTZv: planes per VG ("stencil_z16": 16 -- the ring's refill at the start of
+// every VG and the two z-halo planes are paid per 16 planes instead of 8)
+template <bool kAligned, int kDepth = STENCIL_KD, int kTZv = 8>
 struct StencilT {
   using Args = accel_stencil_args;
   static constexpr int kThreads = 256;
-  static constexpr int kTX = 128, kTY = 8, kTZ = 8;
+  static constexpr int kTX = 128, kTY = 8, kTZ = kTZv;
   static constexpr uint32_t kChunk = 1;
   // the ragged path needs a few more registers; the deep ring (55 KB) fits 4 per SM
   static constexpr int kMinBlocks = (kAligned && kDepth <= 4) ? 5 : 4;
@@ -57,7 +59,7 @@ struct StencilT {
   // "full" completes when all 256 threads' cp.async pieces of the plane landed
   // (cp.async.mbarrier.arrive.noinc), "empty" when all 8 warps released it, so
   // warps drift apart by up to a plane instead of meeting at every plane.
-  static constexpr bool kMbar = STENCIL_MBAR != 0;
+  static constexpr bool kMbar = STENCIL_MBAR != 0 && kTZv + 2 <= 2 * (kDepth + 2);   // (z16: barrier path)
   static_assert(!kMbar || kTZ + 2 <= 2 * kR, "a slot is filled at most twice per VG (parities 0, 1)");
   static constexpr uint32_t kBarBytes = kMbar ? 2 * kR * 8 : 0;
   static constexpr uint32_t kDynSmem = kR * kSlot + kBarBytes + 128;   // + alignment
@@ -201,8 +203,7 @@ struct StencilT {
       mbar_wait(fullb + 8u, 0);
       zm = lds_f4(slot(0) + own);
       cur = lds_f4(slot(1) + own);
-      __syncwarp();
-      if (lane == 0) mbar_arrive(emptyb);   // plane 0 released
+      mbar_release_after(emptyb, __float_as_uint(zm.x), (uint32_t)nz >> 31, lane);   // plane 0 released
     } else {
       // planes 0 and 1 landed (groups 0, 1 of kD + 2 committed)
       asm volatile("cp.async.wait_group %0;" ::"n"(kD) : "memory");
@@ -254,8 +255,8 @@ struct StencilT {
         // plane pz read for the last time (ym, yp, edge): release it; then
         // refill the slot of plane pz-1 (released by every warp after its
         // iteration i-1) with plane pz+kD+1
-        __syncwarp();
-        if (lane == 0) mbar_arrive(emptyb + 8u * (uint32_t)(pz % kR));
+        mbar_release_after(emptyb + 8u * (uint32_t)(pz % kR),
+                           __float_as_uint(ym.x) ^ __float_as_uint(yp.x) ^ __float_as_uint(ev), (uint32_t)nz >> 31, lane);
         if (pz + kD + 1 < nplanes) {
           mbar_wait(emptyb + 8u * (uint32_t)((pz - 1) % kR), 0u);
           issue(pz + kD + 1);
@@ -439,6 +440,7 @@ struct Stencil2T {
 using Stencil = StencilT<true>;
 using StencilX = StencilT<false>;
 using StencilDeep = StencilT<true, 8>;
+using StencilZ16 = StencilT<true, STENCIL_KD, 16>;
 using Stencil2 = Stencil2T<STENCIL2_KD>;
 
 }  // namespace accel

@@ -33,6 +33,13 @@
 
 namespace accel {
 
+// diagnostic build switch (scripts/diag_tma_check.py, diag_tma_which.py):
+// compare every staged plane row with an L2 load (the product build leaves
+// it out: the extra code spilled the 40-register budget)
+#ifndef ACCEL_XP_TMA_DBG
+#define ACCEL_XP_TMA_DBG 0
+#endif
+
 // kBulk: the same ring filled by plain 1-D bulk copies (cp.async.bulk, one
 // per in-volume row segment of a plane) instead of 3-D tensor boxes: no
 // tensor map; rows and columns outside the volume are not copied (their smem
@@ -61,6 +68,12 @@ struct StencilTmaT {
     return __fsub_rn(__fmul_rn(s, c1), __fmul_rn(c, c0));
   }
 
+  // The race behind the drift next to bfs (scripts/diag_tma_which.py): a
+  // consumer warp released a ring slot right after ISSUING its ld.shared of
+  // the slot; the producer, spinning on that empty barrier, issued the TMA of
+  // plane z0+7 into slot 0, which landed before the load read it -- the staged
+  // "plane z0-1" values equalled plane z0+7 exactly.  Slots are now released
+  // with tma::mbar_release_after (the release waits for the loaded data).
   static __device__ __forceinline__ void body(const Args& a, const VirtualBlock& vb, char* smem_raw) {
     using namespace tma;
     const uint32_t r = vb.launch_idx;
@@ -99,7 +112,11 @@ struct StencilTmaT {
         const uint32_t rowb = 4u * (uint32_t)(xe - xs), dcol = 4u * (uint32_t)(xs - (x0 - 4));
         const int ys = max(y0 - 1, 0), ye = min(y0 + kTY + 1, ny);
         const float* in = r == 0 ? a.a0 : ((r & 1u) ? a.buf0 : a.buf1);
-        for (int p = 0; p < nplanes; ++p) {
+        // diagnostics (scripts/diag_tma_check.py): l2hint bit 3 = issue plane 1
+        // before plane 0; bit 4 = wait 2 us after the proxy fence
+        if (a.l2hint & 16u) __nanosleep(2000);
+        for (int p0 = 0; p0 < nplanes; ++p0) {
+          const int p = (a.l2hint & 8u) ? (p0 == 0 ? 1 : (p0 == 1 ? 0 : p0)) : p0;
           if (p >= kNS) mbar_wait(empty(p), (uint32_t)((p / kNS) - 1) & 1u);
           if constexpr (kBulk) {
             const int z = z0 - 1 + p;
@@ -116,11 +133,11 @@ struct StencilTmaT {
             }
           } else {
             mbar_expect_tx(full(p), kPlaneBytes);
-            if (a.l2hint == 0)
+            if ((a.l2hint & 3u) == 0)
               tma_load_3d(slot(p), map, x0 - 4, y0 - 1, z0 - 1 + p, full(p));
             else
               tma_load_3d_hint(slot(p), map, x0 - 4, y0 - 1, z0 - 1 + p, full(p),
-                               a.l2hint == 1 ? policy_evict_first() : policy_evict_last());
+                               (a.l2hint & 3u) == 1 ? policy_evict_first() : policy_evict_last());
           }
         }
       }
@@ -143,10 +160,36 @@ struct StencilTmaT {
     const uint32_t edge = 4u * (uint32_t)((warp + 1) * kCols + (lane == 31 ? 4 + kTX : 3));
     mbar_wait(full(0), 0);
     const float4 zm0 = lds_f4(slot(0) + own);
-    __syncwarp();
-    if (lane == 0) mbar_arrive(empty(0));      // plane z0-1 is only a z neighbour
+    // plane z0-1 is only a z neighbour: release its slot once this warp's
+    // reads of it are ordered before the next TMA into it (release_after)
+    const uint32_t zmask = (uint32_t)nz >> 31;   // 0 at run time (tma::mbar_release_after)
+    mbar_release_after(empty(0), __float_as_uint(zm0.x), zmask, lane);
     mbar_wait(full(1), 0);
     float4 zm = zm0, cur = lds_f4(slot(1) + own);
+    if (ACCEL_XP_TMA_DBG && a.dbg != nullptr) {
+      // diagnostic: the first two planes (z0-1, z0) as staged vs an L2 load (tag 3 << 30: zm, 0 << 30 ... cur)
+      const float* in = r == 0 ? a.a0 : ((r & 1u) ? a.buf0 : a.buf1);
+#pragma unroll
+      for (int s2 = 0; s2 < 2; ++s2) {
+        const int zz = z0 - 1 + s2;
+        const float4 st = s2 == 0 ? zm : cur;
+        if (active && zz >= 0 && zz < nz) {
+          const float4 g = __ldcg(reinterpret_cast<const float4*>(in + ((size_t)zz * ny + y) * nx + x0 + 4 * lane));
+          const float sv[4] = {st.x, st.y, st.z, st.w}, gv[4] = {g.x, g.y, g.z, g.w};
+#pragma unroll
+          for (int e = 0; e < 4; ++e)
+            if (__float_as_uint(sv[e]) != __float_as_uint(gv[e])) {
+              const uint32_t k = atomicAdd(a.dbg, 1u);
+              if (k < 16u) {
+                uint32_t* rec = a.dbg + 8 + 8 * k;
+                rec[0] = r; rec[1] = (uint32_t)zz | (3u << 30); rec[2] = (uint32_t)y;
+                rec[3] = (uint32_t)(x0 + 4 * lane + e); rec[4] = __float_as_uint(sv[e]); rec[5] = __float_as_uint(gv[e]);
+                rec[6] = smid(); rec[7] = (uint32_t)s2;
+              }
+            }
+        }
+      }
+    }
     const long long pstr = (long long)nx * ny;
     float* po = out + ((size_t)z0 * ny + y) * nx + x0 + 4 * lane;
 #pragma unroll 1
@@ -155,11 +198,59 @@ struct StencilTmaT {
       mbar_wait(full(pz + 1), (uint32_t)((pz + 1) / kNS) & 1u);
       const uint32_t P = slot(pz);
       const float4 zp = lds_f4(slot(pz + 1) + own);
+      if (ACCEL_XP_TMA_DBG && a.dbg != nullptr) {
+        // diagnostic: the staged row of plane z0+i+1 vs an L2 load of the same input
+        const int zz = z0 + i + 1;
+        if (active && zz < nz) {
+          const float* in = r == 0 ? a.a0 : ((r & 1u) ? a.buf0 : a.buf1);
+          const float* ot = (r & 1u) ? a.buf1 : a.buf0;
+          const size_t off = ((size_t)zz * ny + y) * nx + x0 + 4 * lane;
+          const float4 g = __ldcg(reinterpret_cast<const float4*>(in + off));
+          const float4 o = __ldcg(reinterpret_cast<const float4*>(ot + off));
+          const float sv[4] = {zp.x, zp.y, zp.z, zp.w}, gv[4] = {g.x, g.y, g.z, g.w}, ov[4] = {o.x, o.y, o.z, o.w};
+#pragma unroll
+          for (int e = 0; e < 4; ++e)
+            if (__float_as_uint(sv[e]) != __float_as_uint(gv[e])) {
+              const uint32_t k = atomicAdd(a.dbg, 1u);
+              if (k < 16u) {
+                uint32_t* rec = a.dbg + 8 + 8 * k;
+                rec[0] = r; rec[1] = (uint32_t)zz; rec[2] = (uint32_t)y; rec[3] = (uint32_t)(x0 + 4 * lane + e);
+                rec[4] = __float_as_uint(sv[e]); rec[5] = __float_as_uint(gv[e]); rec[6] = smid();
+                rec[7] = __float_as_uint(ov[e]);
+              }
+            }
+        }
+      }
       const float4 ym = lds_f4(P + own - 4u * kCols);
       const float4 yp = lds_f4(P + own + 4u * kCols);
       const float ev = lds_f32(P + edge);
-      __syncwarp();
-      if (lane == 0) mbar_arrive(empty(pz));   // plane pz read for the last time
+      if (ACCEL_XP_TMA_DBG && a.dbg != nullptr) {
+        // diagnostic: the y neighbours of plane z0+i as staged vs an L2 load (tag z | 1 << 30: ym, 2 << 30: yp)
+        const int zc = z0 + i;
+        const float* in = r == 0 ? a.a0 : ((r & 1u) ? a.buf0 : a.buf1);
+#pragma unroll
+        for (int s2 = 0; s2 < 2; ++s2) {
+          const int yy = s2 == 0 ? y - 1 : y + 1;
+          const float4 st = s2 == 0 ? ym : yp;
+          if (x0 + 4 * lane < nx && yy >= 0 && yy < ny && zc < nz) {
+            const float4 g = __ldcg(reinterpret_cast<const float4*>(in + ((size_t)zc * ny + yy) * nx + x0 + 4 * lane));
+            const float sv[4] = {st.x, st.y, st.z, st.w}, gv[4] = {g.x, g.y, g.z, g.w};
+#pragma unroll
+            for (int e = 0; e < 4; ++e)
+              if (__float_as_uint(sv[e]) != __float_as_uint(gv[e])) {
+                const uint32_t k = atomicAdd(a.dbg, 1u);
+                if (k < 16u) {
+                  uint32_t* rec = a.dbg + 8 + 8 * k;
+                  rec[0] = r; rec[1] = (uint32_t)zc | ((uint32_t)(s2 + 1) << 30); rec[2] = (uint32_t)yy;
+                  rec[3] = (uint32_t)(x0 + 4 * lane + e); rec[4] = __float_as_uint(sv[e]); rec[5] = __float_as_uint(gv[e]);
+                  rec[6] = smid(); rec[7] = 0xffffffffu;
+                }
+              }
+          }
+        }
+      }
+      // plane pz read for the last time (ym, yp and the edge; zp belongs to plane pz+1)
+      mbar_release_after(empty(pz), __float_as_uint(ym.x) ^ __float_as_uint(yp.x) ^ __float_as_uint(ev), zmask, lane);
       float xl = __shfl_up_sync(0xffffffffu, cur.w, 1);
       float xr = __shfl_down_sync(0xffffffffu, cur.x, 1);
       if (lane == 0) xl = ev;

@@ -36,6 +36,21 @@ __device__ __forceinline__ void mbar_wait(uint32_t bar, uint32_t parity) {
     if (spin > (1ull << 26)) __trap();
   }
 }
+// Release a ring slot (arrive on its "empty" mbarrier) only after this
+// warp's reads of it have RETURNED.  mbarrier.arrive is performed by the
+// barrier unit (SYNCS) and may complete before a preceding ld.shared has read
+// the SRAM; a producer spinning on the barrier can then refill the slot (TMA)
+// under the pending load -- measured on the TMA stencil next to bfs, whose
+// shared-memory atomics slow the loads: the consumer read the plane staged 8
+// slots later (stencil staging).  `loaded` folds bits of the
+// loaded values; zero_mask is 0 at run time but opaque to the compiler (e.g.
+// nz >> 31), so every lane's REDUX operand waits for its loads and lane 0
+// arrives on bar + 0.
+__device__ __forceinline__ void mbar_release_after(uint32_t bar, uint32_t loaded, uint32_t zero_mask, int lane) {
+  const uint32_t all = __reduce_or_sync(0xffffffffu, loaded & zero_mask);
+  if (lane == 0) mbar_arrive(bar + all);
+}
+
 // Loads from a 32-bit shared-window address (keeps the access in the shared
 // state space: a generic pointer rebuilt from an aligned address costs an
 // address-window lookup per access).  volatile: ordered after mbar_wait.

@@ -207,7 +207,8 @@ class StencilJob(Job):
                 self.args.gmaps = self.gmaps.data_ptr()
         self.kernel = kernel
         ty = 16 if kernel == "stencil2" else self.TY   # stencil2: two rows per warp
-        grid = (_cdiv(self.nx, self.TX), _cdiv(self.ny, ty), _cdiv(self.nz, self.TZ))
+        tz = 16 if kernel == "stencil_z16" else self.TZ   # stencil_z16: 16 planes per VG
+        grid = (_cdiv(self.nx, self.TX), _cdiv(self.ny, ty), _cdiv(self.nz, tz))
         self.steps = [Step(kernel, grid, self.args, self.sweeps)]
 
     def result(self):

@@ -86,7 +86,7 @@ def test_mop_small_fullcaps(acc, oracle_lib):
                                        ("tiny", dict(nx=129, ny=8, nz=9, sweeps=2)),    # one column past a tile
                                        ("tiny", dict(nx=2, ny=5, nz=4, sweeps=2)),      # all faces
                                        ("small", dict(sweeps=10))])
-@pytest.mark.parametrize("kernel", ["default", "stencil_tma", "stencil", "stencil2"])
+@pytest.mark.parametrize("kernel", ["default", "stencil_tma", "stencil", "stencil2", "stencil_z16"])
 def test_stencil(acc_tiny_caps, oracle_lib, size, over, kernel):
     """default = the job's choice for this nx; "stencil" (8 rows per tile),
     "stencil2" (16 rows, two per warp) and "stencil_tma" (TMA ring) need
@@ -101,7 +101,7 @@ def test_stencil(acc_tiny_caps, oracle_lib, size, over, kernel):
     assert_close_fp32(sh["a"], oracle_lib.stencil(d), what="stencil")
 
 
-@pytest.mark.parametrize("kernel", ["stencil_tma", "stencil", "stencil2"])
+@pytest.mark.parametrize("kernel", ["stencil_tma", "stencil", "stencil2", "stencil_z16"])
 def test_stencil_default_sampled(acc, oracle_lib, kernel):
     """BASELINE size (512x512x64, 100 sweeps) in the bench's launch
     configuration; the oracle at full size is ~1.7e9 point-sweeps of plain C,
@@ -331,6 +331,8 @@ def _stencil_fp32_replica(d):
                                          ("stencil2", dict(nx=136, ny=17, nz=19, sweeps=4)),
                                          ("stencil2", dict(nx=260, ny=33, nz=8, sweeps=3)),
                                          ("stencil2", dict(nx=4, ny=3, nz=3, sweeps=2)),
+                                         ("stencil_z16", dict(nx=136, ny=17, nz=37, sweeps=4)),
+                                         ("stencil_z16", dict(nx=132, ny=9, nz=16, sweeps=3)),
                                          ("stencil_x", dict(nx=70, ny=21, nz=19, sweeps=3))])
 def test_stencil_bit_exact_fp32_sequence(acc_tiny_caps, kernel, over):
     """Every stencil kernel computes the pinned fp32 round-to-nearest sequence
@@ -393,3 +395,33 @@ def test_tpacf_custom_edges(acc_tiny_caps, oracle_lib, edges):
     dd, rr, dr = oracle_lib.tpacf(d)
     for r in (nat, sh):
         assert np.array_equal(r["dd"], dd) and np.array_equal(r["rr"], rr) and np.array_equal(r["dr"], dr)
+
+
+@pytest.mark.parametrize("kernel", ["stencil_tma", "stencil_bulk"])
+def test_stencil_async_staging_next_to_bfs(acc, kernel):
+    """Regression for the ring-slot race (stencil staging): a
+    consumer warp released a slot before its ld.shared had read it, and next
+    to bfs (whose shared-memory atomics slow those loads) the producer's TMA of
+    a later plane landed first.  The TMA/bulk-staged sweep must equal the
+    cp.async sweep bit for bit (same pinned fp32 op sequence) at the bench's
+    size, next to bfs, in every mode."""
+    from paper_conf_cgo_margiolaso16_b200 import abi
+    from paper_conf_cgo_margiolaso16_b200.jobs import StencilJob, make_job
+    d = synth.preset("stencil", "default", sweeps=12)
+    acc.set_mode(abi.MODE_NATIVE, abi.POLICY_STATIC)
+    ref_job = StencilJob(d, kernel="stencil")
+    acc.run([ref_job])
+    ref = ref_job.result()["a"]
+    bfs = make_job("bfs", synth.preset("bfs", "default"))
+    bfs.fit_levels(acc)
+    try:
+        for mode, pol in [(abi.MODE_NATIVE, abi.POLICY_STATIC), (abi.MODE_SHARED, abi.POLICY_STATIC),
+                          (abi.MODE_SHARED, abi.POLICY_RESOLVE)]:
+            acc.set_mode(mode, pol)
+            for _ in range(2):
+                sj = StencilJob(d, kernel=kernel)
+                acc.run([bfs, sj])
+                got = sj.result()["a"]
+                assert np.array_equal(got, ref), (mode, pol, int((got != ref).sum()))
+    finally:
+        acc.set_mode(abi.MODE_SHARED, abi.POLICY_STATIC)
