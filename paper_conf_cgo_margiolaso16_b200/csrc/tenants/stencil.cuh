@@ -14,11 +14,11 @@
 // shuffles.  Occupancy is set by shared memory (6 CTAs/SM, ~130 KB in flight
 // per SM).  Algorithmic traffic: 8 B per point per sweep.
 //
-// A TMA (cp.async.bulk.tensor.2d) staging of the same tiles was 14 % faster
-// in isolation but returned stale tile data when it ran concurrently with
-// the bfs tenant (boxes partially outside the volume at the x faces; never
-// reproduced in isolation or for the sgemm tenant's in-bounds boxes) -- see
-// DESIGN.md, "stencil staging".
+// The TMA staging of the same tiles (stencil_tma.cuh) once drifted next to
+// the bfs tenant: a ring-slot release raced its own ld.shared (root cause
+// and fix in DESIGN.md, "stencil staging"; tma::mbar_release_after).  Fixed,
+// it is correct but not faster than this cp.async kernel, which stays the
+// default.
 #pragma once
 #include "../device/dispatch.cuh"
 #include "accel_tenants.h"
