@@ -35,9 +35,11 @@
 // host monitor on the tenant's second stream, which serve the current launch
 // and then follow the request's later launches.
 //
-// Completion accounting (who waits for whom).  Launch l+1's main grid and the
-// request's join kernel follow launch l's main grid in stream order
-// (griddepcontrol.wait / the kernel boundary), so they only need launch l's
+// Completion accounting (who waits for whom).  Launch l+1's main grid follows
+// launch l's main grid in stream order (griddepcontrol.wait / the kernel
+// boundary), and so does whatever follows the request's LAST main grid, whose
+// CTAs retire only after that launch's top-ups (kCfgLast: the request's join).
+// So the main grids only need launch l's
 // TOP-UP CTAs to be done: a top-up CTA counts itself in `tu_alive` before it
 // joins a launch and leaves it with a release fence + decrement
 // (wait_topups).  A top-up CTA is in no stream order with the main grids:
@@ -405,6 +407,8 @@ enum : uint32_t {
   kCfgAccount = 1u << 21,  // RESOLVE main grid whose CTAs retire with the fenced `alive`
                            // decrement (a request with an early main grid, R-place-3)
   kCfgTopup = 1u << 22,    // a top-up CTA (accel_topup): always accounts
+  kCfgLast = 1u << 23,     // RESOLVE: the request's last launch -- its main CTAs retire only
+                           // after the launch's top-ups (the request's join, in stream order)
   // measurement-only ablations (env ACCEL_ABLATE on the host; scripts/isolated.py)
   kAblNoFence = 1u << 24,  // retire without the release fence (UNSAFE with top-ups)
   kAblNoLive = 1u << 25,   // never load the live quota (no shrink)
@@ -545,6 +549,13 @@ __device__ __forceinline__ void retire(Desc* d, uint32_t cfg, const SchedState* 
     if (cfg & kCfgTopup) {
       fence_acq_rel();
       atomicSub(&d->tu_alive, 1u);
+    } else if (cfg & kCfgLast) {
+      // the request's join: its last main grid completes only after any
+      // top-up CTAs of that launch (what follows on the tenant stream -- copies
+      // back, the next request -- sees their results).  A top-up that joins
+      // after this check finds the queue dry and writes nothing.
+      fence_acq_rel();
+      if (ld_volatile(&d->topped)) wait_topups(d);
     }
   }
   if (cfg & kCfgStamps) red_max_u64(&d->t_last, globaltimer());

@@ -38,8 +38,6 @@ struct InitParams {
 
 // Fill the descriptors of one request on `s` (one tiny kernel).
 cudaError_t launch_desc_init(const InitParams& p, uint32_t n_desc, cudaStream_t s);
-// RESOLVE: wait (1 thread) until the request's last launch and its top-ups completed.
-cudaError_t launch_join(const Desc* last, cudaStream_t s);
 constexpr size_t kDescBytes = 384;
 // cost-model dequeue order (dispatch.cuh accel_lpt_order): one CTA sorts up to
 // kMaxOrderVGs 64-bit keys in dynamic shared memory

@@ -479,7 +479,8 @@ int enqueue_next(accel_ctx* ctx, Request* r, bool* more) {
     // | kCfgAccount (RESOLVE, a request with an early main grid: its CTAs keep
     // the fenced alive decrement the early grid's wait_complete counts on)
     uint32_t cfg = (k.chunk & 0xffffu) | (resolve ? (1u << 16) : 0u) | (1u << 17) | (li > 0 ? (1u << 18) : 0u) |
-                   (1u << 19) | (resolve && r->early_main ? (1u << 21) : 0u) | ctx->ablate;
+                   (1u << 19) | (resolve && r->early_main ? (1u << 21) : 0u) |
+                   (resolve && li + 1 == r->n_desc ? (1u << 23) : 0u) | ctx->ablate;   // | kCfgLast (the join)
     void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &cfg};
     const dim3 grid = shared ? dim3(st.quota, 1, 1) : dim3(st.grid.x, st.grid.y, st.grid.z);
     const void* fn = shared ? (resolve ? k.prfn : k.pfn) : k.nfn;
@@ -524,7 +525,6 @@ int enqueue_end(accel_ctx* ctx, Request* r) {
     r->enq_li = r->n_desc;   // the early launch was the last one
   }
   if (r->flags & ACCEL_REQ_LAUNCH_EVENTS) CK(ctx, cudaEventRecord(r->ev_launch[r->enq_li], s));
-  if (resolve) CK(ctx, accel::launch_join(ctx->desc_ptr(r->slot + r->n_desc - 1), s));
   for (const accel_copy& c : r->d2h) CK(ctx, cudaMemcpyAsync(c.dst, c.src, c.bytes, cudaMemcpyDeviceToHost, s));
   CK(ctx, cudaEventRecord(r->ev_done, s));
   return ACCEL_OK;

@@ -162,7 +162,7 @@ bool redirect(Wrapped& w, dim3 grid, dim3 block, void** args, size_t smem, cudaS
     return false;
   }
   // the application's later work on its stream waits for the request (its
-  // join kernel on the tenant stream covers RESOLVE growth grids too)
+  // last main grid retires after any RESOLVE growth grids: kCfgLast)
   cudaEventRecord(after, ts);
   cudaStreamWaitEvent(stream, after, 0);
   s.events.push_back(before);   // reusable: recorded and waited on

@@ -69,17 +69,6 @@ __global__ void desc_init_kernel(const InitParams p, uint32_t n_desc) {
   d->qa = st.qa0;
 }
 
-// Request completion: the last launch's main grid precedes this kernel in
-// stream order; wait for its top-up CTAs if a RESOLVE top-up grid joined it.
-__global__ void join_kernel(const Desc* last) {
-  if (threadIdx.x == 0 && ld_volatile(&last->topped)) wait_topups(last);
-}
-
-cudaError_t launch_join(const Desc* last, cudaStream_t s) {
-  join_kernel<<<1, 32, 0, s>>>(last);
-  return cudaGetLastError();
-}
-
 cudaError_t launch_desc_init(const InitParams& p, uint32_t n_desc, cudaStream_t s) {
   const uint32_t threads = 128;
   const uint32_t blocks = (n_desc + threads - 1) / threads;
