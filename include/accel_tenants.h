@@ -68,8 +68,11 @@ typedef struct {
   float *buf1;
   uint32_t nx, ny, nz;
   float c0, c1;
-  uint32_t l2hint;          /* diagnostic: 1 = tensor loads with an L2
-                               evict_first cache policy, 2 = evict_last */
+  uint32_t l2hint;          /* diagnostic: bits 0-1: 1 = tensor loads with
+                               an L2 evict_first cache policy, 2 = evict_last;
+                               bit 3 (8): stage plane 1 before plane 0; bit 4
+                               (16): wait 2 us before the first copy.  0 in
+                               normal use. */
   const accel_tmap *gmaps;  /* diagnostic: non-NULL = read the three maps from
                                this DEVICE array instead of the parameters */
   const float *a0;          /* the input volume (kernel "stencil_bulk": 1-D
