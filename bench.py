@@ -537,10 +537,10 @@ def run_rank(args, rank, world, local, ranks: Ranks) -> dict:
             roof[dom]["traffic"] = tr["dram_bytes_per_launch"]
             roof[dom]["traffic_source"] = tr.get("source")
 
-    # our kernels per step: descriptor init + every launch + the join kernel
-    # (RESOLVE); growth grids come on top (counted from the requests' stats)
-    join = 1 if args.policy != "static" else 0
-    launches_per_step = sum(1 + join + j.launches() for j in jobs)
+    # our kernels per step: descriptor init + every launch (RESOLVE's join is
+    # folded into the last launch); growth grids come on top (counted from the
+    # requests' stats)
+    launches_per_step = sum(1 + j.launches() for j in jobs)
     res = {"rank": rank, "dev_ms": sum(sh["makespan_ms"]), "e2e_ms": sum(ee["makespan_ms"]),
            "nat_ms": sum(na["makespan_ms"]), "oth_ms": {p: sum(v["makespan_ms"]) for p, v in ot.items()},
            "weights": {p: w for p, w in WEIGHTS.items() if w is not None},
