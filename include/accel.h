@@ -125,6 +125,14 @@ typedef struct {
                                  and the rest goes to its co-runners; alone it
                                  keeps its full share.  0 = no cap.  SHARED
                                  only (DESIGN.md R-solver-10). */
+  uint32_t slices;            /* SHARED: run a single launch as this many
+                                 sub-launches over consecutive VG ranges
+                                 (T::kSlices; 0/1 = none).  The sub-launches
+                                 overlap (no dependence between them) and the
+                                 last one retires after all of them, so a
+                                 long persistent request gets fresh CTAs --
+                                 and fresh warp ages -- at every slice
+                                 (DESIGN.md R-disp-9). */
 } accel_kernel_desc;
 
 /* Fill *out with a built-in tenant kernel: "mop", "stencil", "histo", "bfs",

@@ -53,7 +53,7 @@ class accel_kernel_desc(C.Structure):
                 ("topup_fn", vp),
                 ("block", accel_dim3),
                 ("dyn_smem", u32), ("regs", i32), ("chunk", u32), ("args_size", u32), ("order_fn", vp),
-                ("max_ctas_per_sm", u32)]
+                ("max_ctas_per_sm", u32), ("slices", u32)]
 
 
 class accel_kernel_info(C.Structure):

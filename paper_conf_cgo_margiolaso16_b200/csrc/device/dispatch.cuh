@@ -126,12 +126,12 @@ struct alignas(128) Desc {
   Ctl* ctl;              // RESOLVE control block, nullptr otherwise
   uint32_t* coverage;    // verify: coverage[vg] += 1
   uint32_t has_prev;     // this - 1 is the request's previous launch
-  uint32_t pad_a;
+  uint32_t vg_base;      // sliced step (R-disp-9): first VG of this launch's range
   accel_vg_record* trace;  // ACCEL_REQ_TRACE: trace[vg], nullptr otherwise
   uint32_t governed;       // RESOLVE: this launch belongs to the request's main
                            // step, whose CTA count the live quota governs (the
                            // other steps keep their own solved grid)
-  uint32_t pad_b;
+  uint32_t slice;          // sliced step: index of this launch's range (0 = first)
   const uint32_t* order;   // dequeue order (ticket t -> VG order[t]), nullptr = linear
   uint32_t pad0[12];
   // ---- line 1: the software queue head (RUN_TERMINATE when >= total) in the
@@ -263,6 +263,13 @@ struct max_ctas_per_sm : std::integral_constant<uint32_t, 0> {};
 template <class T>
 struct max_ctas_per_sm<T, std::void_t<decltype(T::kMaxCtasPerSm)>>
     : std::integral_constant<uint32_t, (uint32_t)T::kMaxCtasPerSm> {};
+
+// Optional T::kSlices (R-disp-9): SHARED runs of a single launch are split
+// into this many sub-launches over consecutive VG ranges; 0/1 = none.
+template <class T, class = void>
+struct slices_of : std::integral_constant<uint32_t, 1> {};
+template <class T>
+struct slices_of<T, std::void_t<decltype(T::kSlices)>> : std::integral_constant<uint32_t, (uint32_t)T::kSlices> {};
 
 template <class T, class = void>
 struct has_dynamic_total : std::false_type {};
@@ -409,6 +416,9 @@ enum : uint32_t {
   kCfgTopup = 1u << 22,    // a top-up CTA (accel_topup): always accounts
   kCfgLast = 1u << 23,     // RESOLVE: the request's last launch -- its main CTAs retire only
                            // after the launch's top-ups (the request's join, in stream order)
+  kCfgIndep = 1u << 29,    // a later slice of a sliced step: independent of its stream
+                           // predecessor (no griddepcontrol.wait, no predecessor check)
+  kCfgSliceJoin = 1u << 30, // the last slice: its CTAs retire after every earlier slice
   // measurement-only ablations (env ACCEL_ABLATE on the host; scripts/isolated.py)
   kAblNoFence = 1u << 24,  // retire without the release fence (UNSAFE with top-ups)
   kAblNoLive = 1u << 25,   // never load the live quota (no shrink)
@@ -441,6 +451,7 @@ struct SchedState {
   accel_vg_record* trace;
   const uint32_t* order;   // dequeue order of the launch (nullptr: linear / spread)
   Ctl* ctl;                // RESOLVE: the request's control block (d->ctl)
+  uint32_t vg_base;        // sliced step: first VG of this launch's range
   uint32_t governed;       // RESOLVE: the live quota governs this launch
   unsigned long long t0;   // trace: start of the current VG
   // RESOLVE, thread 0: view of the live quota and the admitted count, loaded
@@ -465,11 +476,12 @@ struct SchedState {
   __device__ __forceinline__ void set_cur(uint32_t k, uint32_t vg) {
     cur[k].vg = vg;
     if (vg < total) {
-      uint32_t id = vg;
+      // ticket vg of this launch's range -> VG (vg_base: the range of a slice)
+      uint32_t id = vg_base + vg;
       if (order != nullptr) {
-        id = __ldg(order + vg);
+        id = __ldg(order + vg_base + vg);
       } else if constexpr (kSpread) {
-        id = (uint32_t)(((uint64_t)vg * spread) % total);
+        id = vg_base + (uint32_t)(((uint64_t)vg * spread) % total);
       }
       cur[k].id = id;
       const VirtualBlock b = decode(id, gx, gy, gz, launch_idx);
@@ -557,6 +569,18 @@ __device__ __forceinline__ void retire(Desc* d, uint32_t cfg, const SchedState* 
       fence_acq_rel();
       if (ld_volatile(&d->topped)) wait_topups(d);
     }
+  } else if (cfg & kCfgAccount) {   // STATIC, sliced step: every main CTA accounts
+    fence_acq_rel();
+    atomicAdd(&d->qa, kAliveNeg);
+  }
+  if (cfg & kCfgSliceJoin) {
+    // the last slice completes only after every earlier slice of its step:
+    // they run without a stream dependence (kCfgIndep), and what follows the
+    // step on the stream waits only for this grid.  Their CTAs have all
+    // started (each slice's successor launches once all of them released it),
+    // so this waits on resident CTAs only.
+    const uint32_t n = d->slice;
+    for (uint32_t j = 1; j <= n; ++j) wait_complete(d - j);
   }
   if (cfg & kCfgStamps) red_max_u64(&d->t_last, globaltimer());
 }
@@ -661,6 +685,7 @@ __device__ __forceinline__ void serve(const typename T::Args& args, Desc* d, cha
     S->coverage = d->coverage;
     S->trace = d->trace;
     S->order = d->order;
+    S->vg_base = d->vg_base;
     // descriptor fields the dequeue loop needs, kept in shared memory: a
     // descriptor load there is an L1 miss (and an L2 round trip in front of
     // the dequeue atomic) whenever the tenant's body evicted the line --
@@ -770,7 +795,7 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
 #if ACCEL_XP_PDL == 0
   pdl_release();
 #endif
-  pdl_wait();
+  if (!(cfg & kCfgIndep)) pdl_wait();   // a later slice depends on nothing before it
   serve<T, kResolve>(args, d, smem, &S, cfg, blockIdx.x);
 }
 

@@ -22,6 +22,8 @@ struct InitStep {
   uint64_t qa0;          // initial queue word (alive << 32 | next): main grids with
                          // static first chunks start at grid*chunk (alive = grid
                          // under RESOLVE); 0 otherwise
+  uint32_t slices;       // > 1: a single launch split into this many VG ranges
+  uint32_t slice_vgs;    //      of slice_vgs VGs each (the last may be shorter)
 };
 
 struct InitParams {

@@ -54,6 +54,7 @@ struct Kernel {
   int static_smem;
   int occ_p, occ_n;
   uint32_t max_per_sm;   // useful occupancy cap (0 = none)
+  uint32_t slices;       // R-disp-9: SHARED single launches split into VG ranges (<= 1: none)
   uint32_t threads() const { return block.x * block.y * block.z; }
 };
 
@@ -78,6 +79,8 @@ struct Step {
   uint32_t first;       // first descriptor (relative to the request's slot)
   uint64_t cov_offset;  // coverage offset of the first launch
   const uint32_t* order = nullptr;  // dequeue order (device), nullptr = linear
+  uint32_t slices = 1;     // R-disp-9: > 1 = one launch run as `repeat` VG ranges
+  uint32_t slice_vgs = 0;  //            of slice_vgs VGs
 };
 
 struct Request {
@@ -150,9 +153,9 @@ struct DescHost {
   // line 0
   uint32_t total, gx, gy, gz, chunk, launch_idx, flags, req_idx;
   uint64_t ctl, coverage;
-  uint32_t has_prev, pad_a;
+  uint32_t has_prev, vg_base;
   uint64_t trace;
-  uint32_t governed, pad_b;
+  uint32_t governed, slice;
   uint64_t order;
   uint32_t pad0[12];
   // line 1
@@ -317,10 +320,10 @@ int fetch_result(accel_ctx* ctx, Request* r) {
     CK(ctx, cudaMemcpy(cov.data(), r->cov, cov.size() * sizeof(uint32_t), cudaMemcpyDeviceToHost));
     bool ok = true;
     for (const Step& s : r->steps)
-      for (uint32_t l = 0; l < s.repeat; ++l) {
+      for (uint32_t l = 0; l < (s.slices > 1 ? 1u : s.repeat); ++l) {   // a sliced step: one grid
         const DescHost* d = reinterpret_cast<const DescHost*>(r->desc_host.data() + (size_t)(s.first + l) * kDescBytes);
         // dynamic-total kernels (bfs) cover only the live part of the static grid
-        const uint32_t live = d->total_seen <= s.total ? d->total_seen : s.total;
+        const uint32_t live = s.slices > 1 ? s.total : (d->total_seen <= s.total ? d->total_seen : s.total);
         const uint32_t* c = cov.data() + s.cov_offset + (uint64_t)l * s.total;
         uint32_t bad = 0, first_bad = 0, got = 0;
         for (uint32_t v = 0; v < s.total; ++v) {
@@ -398,11 +401,14 @@ int enqueue_begin(accel_ctx* ctx, Request* r) {
     const Kernel& k = ctx->kernels[st.kid];
     // main grids (SHARED) take static first chunks: the queue head starts
     // past them and, under RESOLVE, every main-grid CTA is admitted
+    // (a sliced step counts its CTAs under both policies: its last slice
+    // waits for the others, R-disp-9)
     const uint64_t qa0 = shared
-        ? ((resolve ? (uint64_t)st.quota << 32 : 0ull) | ((uint64_t)st.quota * k.chunk))
+        ? ((resolve || st.slices > 1 ? (uint64_t)st.quota << 32 : 0ull) | ((uint64_t)st.quota * k.chunk))
         : 0ull;
     p.steps[j] = accel::InitStep{st.first, st.repeat, st.total, st.grid.x, st.grid.y, st.grid.z,
-                                 k.chunk, (uint32_t)st.cov_offset, shared ? st.order : nullptr, qa0};
+                                 k.chunk, (uint32_t)st.cov_offset, shared ? st.order : nullptr, qa0,
+                                 st.slices, st.slice_vgs};
   }
   CK(ctx, accel::launch_desc_init(p, r->n_desc, s));
   if (resolve) {
@@ -478,9 +484,16 @@ int enqueue_next(accel_ctx* ctx, Request* r, bool* more) {
     // | kCfgHasPrev (a request-relative launch precedes this one) | kCfgStaticFirst
     // | kCfgAccount (RESOLVE, a request with an early main grid: its CTAs keep
     // the fenced alive decrement the early grid's wait_complete counts on)
-    uint32_t cfg = (k.chunk & 0xffffu) | (resolve ? (1u << 16) : 0u) | (1u << 17) | (li > 0 ? (1u << 18) : 0u) |
-                   (1u << 19) | (resolve && r->early_main ? (1u << 21) : 0u) |
-                   (resolve && li + 1 == r->n_desc ? (1u << 23) : 0u) | ctx->ablate;   // | kCfgLast (the join)
+    // | kCfgLast (RESOLVE: the request's join).  A sliced step (R-disp-9):
+    // every slice accounts (kCfgAccount), the later ones depend on nothing
+    // before them (kCfgIndep: no predecessor wait, no griddepcontrol.wait),
+    // the last one joins the others (kCfgSliceJoin)
+    const bool sliced = st.slices > 1, indep = sliced && l > 0;
+    uint32_t cfg = (k.chunk & 0xffffu) | (resolve ? (1u << 16) : 0u) | (1u << 17) |
+                   (li > 0 && !indep ? (1u << 18) : 0u) | (1u << 19) |
+                   ((resolve && r->early_main) || sliced ? (1u << 21) : 0u) |
+                   (resolve && li + 1 == r->n_desc ? (1u << 23) : 0u) | (indep ? (1u << 29) : 0u) |
+                   (sliced && l + 1 == st.repeat ? (1u << 30) : 0u) | ctx->ablate;
     void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &cfg};
     const dim3 grid = shared ? dim3(st.quota, 1, 1) : dim3(st.grid.x, st.grid.y, st.grid.z);
     const void* fn = shared ? (resolve ? k.prfn : k.pfn) : k.nfn;
@@ -614,8 +627,17 @@ int build_request(accel_ctx* ctx, const accel_request& in, std::unique_ptr<Reque
     s.quota = s.total;
     s.first = n_desc;
     s.cov_offset = cov;
-    n_desc += L.repeat;
-    cov += (uint64_t)L.repeat * s.total;
+    if (r->mode == ACCEL_MODE_SHARED && k.slices > 1 && L.repeat == 1 && total >= 2ull * k.slices) {
+      // R-disp-9: the launch as `slices` consecutive VG ranges (one coverage region)
+      s.slices = k.slices;
+      s.slice_vgs = (uint32_t)((total + k.slices - 1) / k.slices);
+      s.repeat = (uint32_t)((total + s.slice_vgs - 1) / s.slice_vgs);
+      n_desc += s.repeat;
+      cov += s.total;
+    } else {
+      n_desc += L.repeat;
+      cov += (uint64_t)L.repeat * s.total;
+    }
     r->steps.push_back(std::move(s));
     if (in.main_step < 0 && r->steps.back().total > r->steps[r->main_step].total) r->main_step = (int)j;
   }
@@ -1009,6 +1031,7 @@ int accel_kernel_register(accel_ctx* ctx, const accel_kernel_desc* d, int32_t* k
   k.args_size = d->args_size;
   // ACCEL_NO_OCC_CAP=1: ignore the useful-occupancy caps (A/B measurements)
   k.max_per_sm = std::getenv("ACCEL_NO_OCC_CAP") ? 0u : d->max_ctas_per_sm;
+  k.slices = std::getenv("ACCEL_NO_SLICES") ? 1u : std::max<uint32_t>(1u, d->slices);
   cudaFuncAttributes a;
   CK(ctx, cudaFuncGetAttributes(&a, k.pfn));
   if ((int)k.threads() > a.maxThreadsPerBlock) return ctx->fail(ACCEL_ENOFIT, "block larger than the kernel allows");

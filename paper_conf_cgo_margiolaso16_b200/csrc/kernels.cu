@@ -67,6 +67,18 @@ __global__ void desc_init_kernel(const InitParams p, uint32_t n_desc) {
   d->req_idx = i;
   d->has_prev = i > 0 ? 1u : 0u;
   d->qa = st.qa0;
+  d->vg_base = 0;
+  d->slice = 0;
+  if (st.slices > 1) {
+    // slice r of a single launch (R-disp-9): VGs [r * slice_vgs, ...) of the
+    // same grid; one logical launch (launch_idx 0), one coverage region
+    d->slice = r;
+    d->vg_base = r * st.slice_vgs;
+    d->total = min(st.slice_vgs, st.total - d->vg_base);
+    d->launch_idx = 0;
+    d->coverage = p.coverage ? p.coverage + st.cov_offset : nullptr;
+    d->trace = p.trace ? p.trace + st.cov_offset : nullptr;
+  }
 }
 
 cudaError_t launch_desc_init(const InitParams& p, uint32_t n_desc, cudaStream_t s) {
@@ -90,6 +102,7 @@ accel_kernel_desc make_desc(const char* name) {
   d.chunk = T::kChunk;
   d.args_size = sizeof(typename T::Args);
   d.max_ctas_per_sm = max_ctas_per_sm<T>::value;
+  d.slices = slices_of<T>::value;
   if constexpr (has_vg_cost<T>::value)
     d.order_fn = reinterpret_cast<const void*>(&accel_lpt_order<T>);
   else

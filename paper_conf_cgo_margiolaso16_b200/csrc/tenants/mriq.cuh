@@ -41,6 +41,12 @@ struct MriqQ {
   // CTA per SM nearly saturates the issue slots; its 2nd..6th CTA would take
   // them from a co-runner on the same SM (bfs next to 3 mri-q CTAs/SM: 12x)
   static constexpr uint32_t kMaxCtasPerSm = 1;
+  // R-disp-9: four VG ranges per request in SHARED mode.  mri-q's sin/cos keep
+  // the MUFU pipe busy, and the pipe goes to the OLDER warps: a persistent
+  // mri-q that arrived first starved a later cutcp (rsqrt) for its whole run
+  // (C4; scripts/starve.py).  Fresh CTAs every quarter of the request hand
+  // the age priority back to its co-runners.
+  static constexpr uint32_t kSlices = 4;
   static constexpr uint32_t kDynSmem = 4 * kTile * sizeof(float);
 
   static __device__ __forceinline__ float frac_prod(float k, float x, float& err) {
