@@ -154,3 +154,35 @@ def test_gridding_default(acc, oracle_lib):
     nat, sh, _ = run_modes(acc, lambda: GriddingJob(d))
     same(nat, sh)
     assert_close_fp32(sh["grid"], oracle_lib.gridding(d), what="gridding default")
+
+
+def test_mriq_slices_next_to_cutcp(acc, oracle_lib):
+    """R-disp-9: in SHARED mode mri-q's Q launch runs as 4 VG ranges (1 + 4
+    descriptors; NATIVE keeps 1 + 1), every VG exactly once (the fixture
+    verifies coverage), results as the oracle, under both policies and with
+    a cutcp request submitted while it runs (the co-runner it used to
+    starve)."""
+    import time
+    from paper_conf_cgo_margiolaso16_b200 import abi
+    from paper_conf_cgo_margiolaso16_b200.jobs import MriqJob, make_job
+    d = synth.preset("mriq", "small")
+    pm, qr, qi = oracle_lib.mriq(d)
+    cut = make_job("cutcp", synth.preset("cutcp", "small"))
+    try:
+        for mode, pol, want in [(abi.MODE_NATIVE, abi.POLICY_STATIC, 2), (abi.MODE_SHARED, abi.POLICY_STATIC, 5),
+                                (abi.MODE_SHARED, abi.POLICY_RESOLVE, 5)]:
+            acc.set_mode(mode, pol)
+            job = MriqJob(d)
+            ids = acc.submit([job], tenants=[0])
+            time.sleep(2e-4)
+            ids += acc.submit([cut], tenants=[1])
+            acc.sync()
+            st = [acc.stats(i) for i in ids]
+            acc.release()
+            assert st[0].launches == want, (mode, pol, st[0].launches)
+            assert st[0].coverage_ok == 1 and st[1].coverage_ok == 1
+            res = job.result()
+            assert np.array_equal(res["phimag"], pm)
+            assert_close_fp32(np.concatenate([res["qr"], res["qi"]]), np.concatenate([qr, qi]), what="mri-q sliced")
+    finally:
+        acc.set_mode(abi.MODE_SHARED, abi.POLICY_STATIC)
