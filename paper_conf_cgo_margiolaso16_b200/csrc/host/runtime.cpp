@@ -1032,6 +1032,12 @@ int accel_kernel_register(accel_ctx* ctx, const accel_kernel_desc* d, int32_t* k
   // ACCEL_NO_OCC_CAP=1: ignore the useful-occupancy caps (A/B measurements)
   k.max_per_sm = std::getenv("ACCEL_NO_OCC_CAP") ? 0u : d->max_ctas_per_sm;
   k.slices = std::getenv("ACCEL_NO_SLICES") ? 1u : std::max<uint32_t>(1u, d->slices);
+  if (const char* e = std::getenv("ACCEL_SLICES")) {   // experiment: "name:n,name:n"
+    const std::string spec(e), key = k.name + ":";
+    const size_t at = spec.find(key);
+    if (at != std::string::npos && (at == 0 || spec[at - 1] == ','))
+      k.slices = std::max<uint32_t>(1u, (uint32_t)std::atoi(spec.c_str() + at + key.size()));
+  }
   cudaFuncAttributes a;
   CK(ctx, cudaFuncGetAttributes(&a, k.pfn));
   if ((int)k.threads() > a.maxThreadsPerBlock) return ctx->fail(ACCEL_ENOFIT, "block larger than the kernel allows");
