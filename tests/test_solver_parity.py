@@ -124,3 +124,22 @@ def test_weighted_metrics_equal():
         wu, ws = abi.accel_metrics_weighted(ta, ts, w)
         assert wu == pytest.approx(M.weighted_unfairness(ts, ta, w), rel=1e-12)
         assert ws == pytest.approx(M.weighted_slowdown(ts, ta, w), rel=1e-12)
+
+
+def test_solve_memo_consistent():
+    """accel_solve memoises by (caps, demands) (solver.cpp): a repeated
+    instance -- with other instances solved in between -- returns its first
+    answer, which equals the oracle."""
+    r = random.Random(77)
+    caps = S.Caps(sms=6)
+    inst = []
+    while len(inst) < 8:
+        try:
+            inst.append(_random_instance(r, caps, 4, 40))
+        except S.NoFit:
+            continue
+    first = [abi.accel_solve([_to_c(d) for d in ds], _caps(caps)) for ds in inst]
+    again = [abi.accel_solve([_to_c(d) for d in ds], _caps(caps)) for ds in reversed(inst)][::-1]
+    assert first == again
+    for ds, q in zip(inst, first):
+        assert q == S.solve(ds, caps)
