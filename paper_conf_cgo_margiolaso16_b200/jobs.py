@@ -553,11 +553,16 @@ class HistoPipelineJob(Job):
     (raw samples -> bin indices), then `iters` launches of the main+final
     kernel on the bin stream -- one request, three steps (main = the last)."""
 
-    PER_VG = 16384
+    # samples per VG of the prescan and intermediates steps: 4096 gives 4096
+    # VGs for 2^24 samples, several waves over the persistent grid (16384
+    # left 1024 VGs for 888 CTAs: a second wave of 136 -- +3.9 % STATIC; sweep
+    # in profiles/r2b/histo_pipeline_per_vg.log)
+    PER_VG = 4096
 
     def __init__(self, d: dict, device="cuda"):
         super().__init__(name="histo_pipeline", device=torch.device(device))
         self.n, self.bins, self.iters = d["n"], d["bins"], d["iters"]
+        self.PER_VG = int(d.get("per_vg", os.environ.get("ACCEL_HISTO_PRE_PER_VG", self.PER_VG)))
         self.inputs = {"raw": _dev(d["raw"], self.device)}
         self.bin_stream = torch.empty(self.n, dtype=torch.int32, device=self.device)
         self.lo = torch.empty(1, dtype=torch.int32, device=self.device)
