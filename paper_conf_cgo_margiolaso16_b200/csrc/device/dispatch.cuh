@@ -804,13 +804,20 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
 // the step's later launches (each only once its predecessor completed).
 template <class T>
 __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
-    accel_topup(const __grid_constant__ typename T::Args args, Desc* __restrict__ d, uint32_t sticky) {
+    accel_topup(const __grid_constant__ typename T::Args args, Desc* __restrict__ d, uint32_t sticky_word) {
   extern __shared__ __align__(128) char smem[];
   __shared__ SchedState S;
   __shared__ uint32_t s_l, s_go;
+  // kStickyMain: this grid IS the request's main step (ACCEL_STICKY_MAIN,
+  // experiment): one long-lived grid serves every launch of the step, so its
+  // warps age like a single-launch kernel's instead of being the youngest on
+  // their SM at every launch
+  constexpr uint32_t kStickyMain = 1u << 31;
+  const bool main_grid = (sticky_word & kStickyMain) != 0u;
+  const uint32_t sticky = sticky_word & ~kStickyMain;
   if (threadIdx.x == 0) {
     const uint32_t cur = ld_volatile(&d->ctl->cur);
-    s_l = cur > d->req_idx ? cur - d->req_idx : 0u;
+    s_l = main_grid ? 0u : (cur > d->req_idx ? cur - d->req_idx : 0u);
   }
   __syncthreads();
   for (uint32_t l = s_l; l < sticky; ++l) {
@@ -825,6 +832,10 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
         atomicExch(&dl->topped, 1u);
         atomicAdd(&dl->tu_alive, 1u);   // before the admission atomic (wait_topups)
         fence_acq_rel();
+        // the main grid announces the launch it serves (after launch l-1
+        // completed, so `cur >= l` still implies that for wait_hybrid)
+        if (main_grid)
+          asm volatile("red.release.gpu.global.max.u32 [%0], %1;" ::"l"(&dl->ctl->cur), "r"(dl->req_idx) : "memory");
       }
     }
     __syncthreads();
@@ -838,6 +849,9 @@ __global__ void __launch_bounds__(T::kThreads, min_blocks<T>::value)
     // launches (the monitor tops up afresh on a later growth, apply_quota)
     if (S.over || S.draining) return;
   }
+  // the main grid completes only after every CTA (its own and growth grids')
+  // left the step's last launch: what follows on the stream sees all results
+  if (main_grid && threadIdx.x == 0) wait_topups(d + sticky - 1);
 }
 
 // ---------------------------------------------------------------------------

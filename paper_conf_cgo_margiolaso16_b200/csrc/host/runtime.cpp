@@ -81,6 +81,7 @@ struct Step {
   const uint32_t* order = nullptr;  // dequeue order (device), nullptr = linear
   uint32_t slices = 1;     // R-disp-9: > 1 = one launch run as `repeat` VG ranges
   uint32_t slice_vgs = 0;  //            of slice_vgs VGs
+  bool sticky_main = false;  // ACCEL_STICKY_MAIN experiment: one grid serves every launch
 };
 
 struct Request {
@@ -396,6 +397,11 @@ int enqueue_begin(accel_ctx* ctx, Request* r) {
   p.trace = r->trace;
   p.flags = kFlagStamps | (shared ? kFlagAlive : 0u);
   p.n_steps = (uint32_t)r->steps.size();
+  static const bool sticky_env = std::getenv("ACCEL_STICKY_MAIN") != nullptr;
+  for (size_t j = 0; j < r->steps.size(); ++j) {
+    Step& st = r->steps[j];
+    st.sticky_main = sticky_env && resolve && (int)j == r->main_step && st.repeat > 1 && st.slices <= 1;
+  }
   for (size_t j = 0; j < r->steps.size(); ++j) {
     const Step& st = r->steps[j];
     const Kernel& k = ctx->kernels[st.kid];
@@ -403,8 +409,8 @@ int enqueue_begin(accel_ctx* ctx, Request* r) {
     // past them and, under RESOLVE, every main-grid CTA is admitted
     // (a sliced step counts its CTAs under both policies: its last slice
     // waits for the others, R-disp-9)
-    const uint64_t qa0 = shared
-        ? ((resolve || st.slices > 1 ? (uint64_t)st.quota << 32 : 0ull) | ((uint64_t)st.quota * k.chunk))
+    const uint64_t qa0 = st.sticky_main ? 0ull   // every CTA joins through the queue word
+        : shared ? ((resolve || st.slices > 1 ? (uint64_t)st.quota << 32 : 0ull) | ((uint64_t)st.quota * k.chunk))
         : 0ull;
     p.steps[j] = accel::InitStep{st.first, st.repeat, st.total, st.grid.x, st.grid.y, st.grid.z,
                                  k.chunk, (uint32_t)st.cov_offset, shared ? st.order : nullptr, qa0,
@@ -476,6 +482,20 @@ int enqueue_next(accel_ctx* ctx, Request* r, bool* more) {
   const Step& st = r->steps[r->enq_step];
   const Kernel& k = ctx->kernels[st.kid];
   const uint32_t li = r->enq_li;
+  if (st.sticky_main) {
+    // ACCEL_STICKY_MAIN: one grid of `quota` CTAs serves the step's launches
+    // in order (accel_topup with the main-grid flag)
+    for (uint32_t l = 0; lev && l < st.repeat; ++l) CK(ctx, cudaEventRecord(r->ev_launch[li + l], s));
+    accel::Desc* d = ctx->desc_ptr(r->slot + st.first);
+    uint32_t sticky = st.repeat | (1u << 31);
+    void* params[3] = {const_cast<unsigned char*>(st.args.data()), &d, &sticky};
+    CK(ctx, cudaLaunchKernel(k.tfn, dim3(st.quota, 1, 1), k.block, params, k.dyn_smem, s));
+    r->enq_li += st.repeat;
+    r->enq_launch = 0;
+    r->enq_step += 1;
+    *more = r->enq_step < (r->early_main ? (size_t)r->main_step : r->steps.size());
+    return ACCEL_OK;
+  }
   if (lev) CK(ctx, cudaEventRecord(r->ev_launch[li], s));
   {
     const uint32_t l = r->enq_launch;
