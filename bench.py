@@ -365,6 +365,32 @@ def stub_rank(args, rank, world, ranks: Ranks) -> dict:
 
 
 # ----------------------------------------------------------------- GPU leg
+def size_matched_copy(nbytes: float, roof: dict, reps: int = 20) -> dict:
+    """Context for an HBM-bound kernel's frac: the bandwidth a plain device
+    copy reaches on the SAME bytes per launch (nbytes/2 read + nbytes/2
+    written, back to back, CUDA events).  At ~30 us per launch a copy itself
+    stays well below the large-copy peak (ramp-up and tail of every launch);
+    scripts/stencil_size.py shows the stencil kernel at 0.87 of peak on
+    volumes 8x the default.  Outside the timed region; torch's copy kernel is
+    the yardstick, not part of the path."""
+    import torch
+    n = max(1, int(nbytes // 8))
+    x = torch.ones(n, dtype=torch.float32, device="cuda")
+    y = torch.empty_like(x)
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    for _ in range(3):
+        y.copy_(x)
+    e0.record()
+    for _ in range(reps):
+        y.copy_(x)
+        x, y = y, x
+    e1.record()
+    torch.cuda.synchronize()
+    gbs = 8.0 * n / (e0.elapsed_time(e1) * 1e-3 / reps) / 1e9
+    return {"copy_gbs": gbs, "copy_frac_of_peak": gbs / roof["peak"],
+            "frac": roof["achieved"] / gbs, "isolated_frac": roof["isolated"]["achieved"] / gbs}
+
+
 def run_rank(args, rank, world, local, ranks: Ranks) -> dict:
     """Everything one GPU does: correctness pass, T(a) calibration, the timed
     SHARED steps (barrier + synchronize on both sides), NATIVE and the other
@@ -536,6 +562,9 @@ def run_rank(args, rank, world, local, ranks: Ranks) -> dict:
         if tr:
             roof[dom]["traffic"] = tr["dram_bytes_per_launch"]
             roof[dom]["traffic_source"] = tr.get("source")
+    if dom is not None and roof[dom]["bound"] == "hbm":
+        roof[dom]["size_matched_copy"] = size_matched_copy(works[dom].get("bytes_per_launch", works[dom].get("bytes")),
+                                                           roof[dom])
 
     # our kernels per step: descriptor init + every launch (RESOLVE's join is
     # folded into the last launch); growth grids come on top (counted from the
