@@ -36,7 +36,12 @@ struct Cutcp {
   static constexpr int kMinBlocks = CUTCP_MINB;
   static constexpr int kTile = 128;  // atoms staged per round
   static constexpr int kPts = 4;     // points per thread along z
-  static constexpr uint32_t kDynSmem = kTile * sizeof(float4);
+#ifndef CUTCP_GATHER
+#define CUTCP_GATHER 1
+#endif
+  // tile + (CUTCP_GATHER) per-batch row starts, prefix sums and warp totals
+  static constexpr uint32_t kDynSmem =
+      kTile * sizeof(float4) + (CUTCP_GATHER ? (2 * kThreads + 1 + kThreads / 32) * sizeof(int) : 0);
 
   // MUFU.RSQ without the denormal rescaling rsqrtf() wraps around it (4
   // instructions per in-range pair): r^2 < 2^-126 only occurs for excluded
@@ -136,6 +141,78 @@ struct Cutcp {
       }
     };
     int fill = 0;   // atoms staged in the tile (uniform)
+#if CUTCP_GATHER
+    // The cell rows' atom ranges are found in parallel, one row per thread
+    // per batch of kThreads rows (same (cz, cy) order and fp32 arithmetic as
+    // the row loop below), prefix-summed, and the tile is then gathered one
+    // atom per thread, each locating its row by binary search.  One dependent
+    // global round trip per tile instead of two per row: the tile holds the
+    // same atoms in the same order, so the sums are bit-identical.
+    int* row_a0 = reinterpret_cast<int*>(smem + kTile * sizeof(float4));
+    int* row_pre = row_a0 + kThreads;              // kThreads + 1 entries
+    int* wsum = row_pre + kThreads + 1;            // kThreads / 32 entries
+    const int nyc = cy1 - cy0 + 1, nrows = (cz1 - cz0 + 1) * nyc;
+    for (int rb = 0; rb < nrows; rb += kThreads) {
+      int a0 = 0, len = 0;
+      const int rr = rb + t;
+      if (rr < nrows) {
+        const int cz = cz0 + rr / nyc, cy = cy0 + rr % nyc;
+        const float gz = gap(bz0, bz1, cz * cs, (cz + 1) * cs);
+        const float gy = gap(by0, by1, cy * cs, (cy + 1) * cs);
+        const float d2 = gy * gy + gz * gz;
+        if (d2 < cm * cm) {
+          const float rx = sqrtf(cm * cm - d2);
+          const int cx0 = clampc((int)floorf((bx0 - rx) / cs)), cx1 = clampc((int)floorf((bx1 + rx) / cs));
+          const int row = (cz * nc + cy) * nc;
+          a0 = __ldg(a.cell_start + row + cx0);
+          len = __ldg(a.cell_start + row + cx1 + 1) - a0;
+        }
+      }
+      // block exclusive scan of len
+      int inc = len;
+#pragma unroll
+      for (int o = 1; o < 32; o <<= 1) {
+        const int v = __shfl_up_sync(0xffffffffu, inc, o);
+        if ((t & 31) >= o) inc += v;
+      }
+      __syncthreads();   // the previous batch's gather is done with row_a0 / row_pre
+      if ((t & 31) == 31) wsum[t >> 5] = inc;
+      __syncthreads();
+      int base = 0, tot = 0;
+#pragma unroll
+      for (int w = 0; w < kThreads / 32; ++w) {
+        const int s = wsum[w];
+        base += w < (t >> 5) ? s : 0;
+        tot += s;
+      }
+      row_a0[t] = a0;
+      row_pre[t] = base + inc - len;
+      if (t == 0) row_pre[kThreads] = tot;
+      __syncthreads();
+      for (int done = 0; done < tot;) {
+        const int take = min(kTile - fill, tot - done);
+        if (t < take) {
+          const int pos = done + t;
+          // the last row r with row_pre[r] <= pos: never an empty row (its
+          // successor starts at the same position); row_pre[kThreads] = tot > pos
+          int lo = 0, hi = kThreads;
+          while (hi - lo > 1) {
+            const int mid = (lo + hi) >> 1;
+            if (row_pre[mid] <= pos) lo = mid; else hi = mid;
+          }
+          tile[fill + t] = __ldg(reinterpret_cast<const float4*>(a.atoms) + row_a0[lo] + (pos - row_pre[lo]));
+        }
+        fill += take;
+        done += take;
+        if (fill == kTile) {
+          __syncthreads();
+          evaluate(kTile);
+          __syncthreads();
+          fill = 0;
+        }
+      }
+    }
+#else
     for (int cz = cz0; cz <= cz1; ++cz) {
       const float gz = gap(bz0, bz1, cz * cs, (cz + 1) * cs);
       for (int cy = cy0; cy <= cy1; ++cy) {
@@ -161,6 +238,7 @@ struct Cutcp {
         }
       }
     }
+#endif
     if (fill) {
       __syncthreads();
       evaluate(fill);
