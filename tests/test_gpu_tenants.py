@@ -232,7 +232,10 @@ def test_bfs_default(acc, oracle_lib):
 
 
 # ---------------------------------------------------------------- cutcp
-@pytest.mark.parametrize("size,over", [("tiny", {}), ("tiny", dict(seed=5, box=24.0)), ("small", {})])
+# default 1-A cells: ~290 cell rows per VG, three gather batches of 128 rows;
+# 4-A and 2-A cells: one batch, longer rows (the row gather, cutcp.cuh)
+@pytest.mark.parametrize("size,over", [("tiny", {}), ("tiny", dict(seed=5, box=24.0)), ("small", {}),
+                                       ("tiny", dict(cell=4.0)), ("small", dict(seed=2, cell=2.0))])
 def test_cutcp(acc_tiny_caps, oracle_lib, size, over):
     from paper_conf_cgo_margiolaso16_b200.jobs import CutcpJob
     d = synth.preset("cutcp", size, **over)
