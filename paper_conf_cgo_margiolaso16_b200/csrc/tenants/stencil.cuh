@@ -45,7 +45,10 @@ struct StencilT {
   static constexpr int kTX = 128, kTY = 8, kTZ = kTZv;
   static constexpr uint32_t kChunk = 1;
   // the ragged path needs a few more registers; the deep ring (55 KB) fits 4 per SM
-  static constexpr int kMinBlocks = (kAligned && kDepth <= 4) ? 5 : 4;
+#ifndef STENCIL_MINB
+#define STENCIL_MINB 5
+#endif
+  static constexpr int kMinBlocks = (kAligned && kDepth <= 4) ? STENCIL_MINB : 4;
   static constexpr int kRows = kTY + 2;                 // y halo
   static constexpr int kCols = kTX + 8;                 // x0-4 .. x0+131 (16-B multiples)
   static constexpr uint32_t kPlaneBytes = kRows * kCols * 4;          // 5440
